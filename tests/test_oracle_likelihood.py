@@ -1,0 +1,190 @@
+"""Pins of the oracle's model and data likelihood.
+
+Each pin fixes the oracle against something other than itself: known-answer
+vectors, the matrix exponential of the F81 rate matrix, brute-force summation
+over all ancestral states, closed forms and invariances.
+"""
+import itertools
+
+import numpy as np
+import pytest
+import scipy.linalg
+
+import synth
+
+
+# ------------------------------------------------------------------ P17 RNG
+def test_philox_known_answers(orc):
+    # Random123 kat_vectors for philox4x32_10 (Salmon et al., SC'11)
+    kat = [
+        ([0, 0, 0, 0], [0, 0], [0x6627E8D5, 0xE169C58D, 0xBC57AC4C, 0x9B00DBD8]),
+        ([0xFFFFFFFF] * 4, [0xFFFFFFFF] * 2, [0x408F276D, 0x41C83B0E, 0xA20BC7C6, 0x6D5451FD]),
+        ([0x243F6A88, 0x85A308D3, 0x13198A2E, 0x03707344], [0xA4093822, 0x299F31D0],
+         [0xD16CFE09, 0x94FDCCEB, 0x5001E420, 0x24126EA1]),
+    ]
+    for ctr, key, want in kat:
+        assert list(orc.philox(ctr, key)) == want
+
+
+def test_u01_range_and_resolution(orc):
+    lib = orc.lib()
+    assert lib.orc_u01(0, 0) == 2.0 ** -53
+    assert lib.orc_u01(0xFFFFFFFF, 0xFFFFFFFF) == 1.0
+    us = np.array([orc.uniform(7, 3, s, 1, i) for s in range(50) for i in range(40)])
+    assert us.min() > 0.0 and us.max() <= 1.0
+    assert abs(us.mean() - 0.5) < 0.02
+
+
+# ------------------------------------------------------------------ P1 F81
+def _f81_Q(pi, u):
+    Q = u * np.tile(pi, (4, 1))
+    np.fill_diagonal(Q, 0.0)
+    np.fill_diagonal(Q, -Q.sum(axis=1))
+    return Q
+
+
+@pytest.mark.parametrize("pi", [[0.25] * 4, [0.1, 0.2, 0.3, 0.4], [0.7, 0.1, 0.1, 0.1]])
+def test_transition_is_expm_of_f81_generator(orc, pi):
+    pi = np.array(pi)
+    u = orc.default_rate(pi)
+    assert np.isclose(u, 1.0 / (1.0 - np.sum(pi ** 2)))
+    Q = _f81_Q(pi, u)
+    for t in [0.0, 1e-9, 0.01, 0.3, 2.0, 40.0]:
+        P = orc.transition(t, u, pi)
+        assert np.allclose(P, scipy.linalg.expm(Q * t), rtol=1e-12, atol=1e-14)
+        assert np.allclose(P.sum(axis=1), 1.0, atol=1e-15)
+    assert np.array_equal(orc.transition(0.0, u, pi), np.eye(4))
+    assert np.allclose(orc.transition(1e6, u, pi), np.tile(pi, (4, 1)), atol=1e-15)
+    # Chapman-Kolmogorov
+    P1, P2, P12 = (orc.transition(t, u, pi) for t in (0.2, 0.45, 0.65))
+    assert np.allclose(P1 @ P2, P12, atol=1e-15)
+    # expected substitutions per unit time equal 1 under u = 1/(1 - sum pi^2) (reading S3)
+    assert np.isclose(-np.dot(pi, np.diag(Q)), 1.0)
+
+
+# ------------------------------------------------------------------ P3 brute force
+def _brute_force_loglik(codes, parent, age, pi, u):
+    """Sum over all 4^(n-1) interior assignments of pi_root * prod_branches P."""
+    n = codes.shape[0]
+    nn = 2 * n - 1
+    root = int(np.where(parent < 0)[0][0])
+    Q = _f81_Q(pi, u)
+    Pb = {v: scipy.linalg.expm(Q * (age[parent[v]] - age[v])) for v in range(nn) if parent[v] >= 0}
+    interior = list(range(n, nn))
+    total = np.zeros(codes.shape[1])
+    for assign in itertools.product(range(4), repeat=len(interior)):
+        state = {v: a for v, a in zip(interior, assign)}
+        prob = np.full(codes.shape[1], pi[state[root]])
+        for v in range(nn):
+            if parent[v] < 0:
+                continue
+            ps = state[parent[v]]
+            if v < n:
+                prob = prob * Pb[v][ps, codes[v]]
+            else:
+                prob = prob * Pb[v][ps, state[v]]
+        total += prob
+    return np.log(total)
+
+
+@pytest.mark.parametrize("n", [2, 3, 4, 5])
+@pytest.mark.parametrize("shape", ["caterpillar", "balanced", "random"])
+def test_pruning_equals_brute_force(orc, n, shape):
+    rng = np.random.default_rng(100 + n)
+    parent, age = synth.shaped_tree(n, shape, rng, scale=0.3)
+    pi = np.array([0.1, 0.2, 0.3, 0.4])
+    u = orc.default_rate(pi)
+    codes = synth.random_alignment(n, 30, rng, pi)
+    ll, site = orc.log_likelihood(codes, parent, age, pi, u, site_ll=True)
+    want = _brute_force_loglik(codes, parent, age, pi, u)
+    assert np.allclose(site, want, rtol=1e-12, atol=1e-12)
+    assert np.isclose(ll, want.sum(), rtol=1e-13)
+
+
+# ------------------------------------------------------------------ P2 / P4 / P5 / P6 / P7
+def test_monomorphic_and_infinite_branches(orc):
+    rng = np.random.default_rng(3)
+    parent, age = synth.shaped_tree(6, "random", rng)
+    codes = np.zeros((6, 25), np.uint8)
+    assert orc.log_likelihood(codes, parent, age, np.array([1.0, 0, 0, 0]), 1.0) == 0.0
+    # infinite branches: every tip independent draw from pi
+    pi = np.array([0.4, 0.3, 0.2, 0.1])
+    codes = synth.random_alignment(6, 25, rng, pi)
+    far = age * 1e4
+    want = np.log(pi[codes]).sum()
+    assert np.isclose(orc.log_likelihood(codes, parent, far, pi, orc.default_rate(pi)), want,
+                      rtol=1e-12)
+
+
+def test_two_tip_pulley_closed_form(orc):
+    pi = np.array([0.3, 0.2, 0.1, 0.4])
+    u = orc.default_rate(pi)
+    parent = np.array([2, 2, -1])
+    age = np.array([0.0, 0.0, 0.37])
+    codes = np.array([[0, 1, 2, 3, 0, 3], [0, 2, 2, 1, 3, 3]], np.uint8)
+    P = scipy.linalg.expm(_f81_Q(pi, u) * 0.74)
+    want = np.sum(np.log(pi[codes[0]] * P[codes[0], codes[1]]))
+    assert np.isclose(orc.log_likelihood(codes, parent, age, pi, u), want, rtol=1e-13)
+
+
+def test_root_position_invariance(orc):
+    # (tip0, (tip1, tip2)v) with the root slid along the root-to-tip0 / root-to-v path
+    pi = np.array([0.25, 0.25, 0.3, 0.2])
+    u = orc.default_rate(pi)
+    rng = np.random.default_rng(5)
+    codes = synth.random_alignment(3, 40, rng, pi)
+    parent = np.array([4, 3, 3, 4, -1])
+    base = orc.log_likelihood(codes, parent, np.array([0.0, 0.0, 0.0, 0.2, 0.5]), pi, u)
+    for d in [-0.15, 0.07, 0.3]:
+        age = np.array([2 * d, 0.0, 0.0, 0.2, 0.5 + d])
+        assert np.isclose(orc.log_likelihood(codes, parent, age, pi, u), base, rtol=1e-12)
+
+
+def test_site_and_label_permutation_and_duplication(orc):
+    rng = np.random.default_rng(11)
+    n = 7
+    parent, age = synth.coalescent_tree(n, 1.0, rng)
+    pi = np.array([0.2, 0.3, 0.3, 0.2])
+    u = orc.default_rate(pi)
+    codes = synth.f81_alignment(parent, age, 64, pi, u, rng)
+    base = orc.log_likelihood(codes, parent, age, pi, u)
+    perm = rng.permutation(64)
+    assert np.isclose(orc.log_likelihood(codes[:, perm], parent, age, pi, u), base, rtol=1e-13)
+    dup = np.concatenate([codes, codes], axis=1)
+    assert np.isclose(orc.log_likelihood(dup, parent, age, pi, u), 2 * base, rtol=1e-13)
+    # relabel tips: tip i -> sigma(i), rows permuted accordingly
+    sigma = rng.permutation(n)
+    parent2 = parent.copy()
+    for i in range(n):
+        parent2[sigma[i]] = parent[i]
+    codes2 = np.zeros_like(codes)
+    codes2[sigma] = codes
+    assert np.isclose(orc.log_likelihood(codes2, parent2, age, pi, u), base, rtol=1e-13)
+
+
+def test_all_zero_branches(orc):
+    n = 5
+    parent = np.array([5, 5, 6, 7, 7, 6, 8, 8, -1], np.int32)
+    age = np.zeros(9)
+    pi = np.array([0.1, 0.2, 0.3, 0.4])
+    const = np.tile(np.array([[0, 3, 2, 2, 1]], np.uint8), (n, 1))
+    assert np.isclose(orc.log_likelihood(const, parent, age, pi, 1.0), np.log(pi[[0, 3, 2, 2, 1]]).sum())
+    mixed = const.copy()
+    mixed[2, 1] = 0
+    assert orc.log_likelihood(mixed, parent, age, pi, 1.0) == -np.inf
+
+
+def test_theta_independence_of_data_likelihood(orc):
+    """Eq. 23 (L720-723): the likelihood has no theta argument; only u and t enter."""
+    rng = np.random.default_rng(2)
+    parent, age = synth.coalescent_tree(5, 0.5, rng)
+    pi = np.full(4, 0.25)
+    codes = synth.f81_alignment(parent, age, 50, pi, 4 / 3, rng)
+    a = orc.log_likelihood(codes, parent, age, pi, 4 / 3)
+    b = orc.log_likelihood(codes, parent, age * 2, pi, 4 / 6)   # (u, t) -> (u/2, 2t)
+    assert np.isclose(a, b, rtol=1e-13)
+
+
+def test_base_freqs_pooled(orc):
+    codes = np.array([[0, 0, 1, 2], [3, 3, 3, 0]], np.uint8)
+    assert np.allclose(orc.base_freqs(codes), [3 / 8, 1 / 8, 1 / 8, 3 / 8])
