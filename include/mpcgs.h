@@ -1,0 +1,205 @@
+/*
+ * mpcgs.h -- C ABI of the B200 (sm_100a) hot path of the multiple-proposal
+ * coalescent genealogy sampler (mpcgs) of P. E. Davis, "Scalable
+ * Parallelization of a Markov Coalescent Genealogy Sampler" (2016).
+ * Citations "L<a>-<b>" are lines of that paper's PAPER.md; readings S1..S23 are
+ * listed in DESIGN.md.
+ *
+ * The library runs one generalized Metropolis-Hastings (GMH) step per call of
+ * its step loop (Alg. 1, Fig. 12):
+ *   target draw (4.3 L1079-1093) -> neighbourhood context (4.2 L986-1027) ->
+ *   N resimulated proposals (4.2 L1028-1043) -> Felsenstein pruning data
+ *   likelihood under F81 (Eq. 19-22) -> weights over N+1 states
+ *   (Eq. 29-31) and inverse-CDF draws (L1140-1144),
+ * and, after sampling, maximises the relative likelihood L(theta)/L(theta0)
+ * (Eq. 25-26, 5.1.5 L1306-1311).
+ *
+ * Conventions (all entry points):
+ *  - Every function returning mpcgs_status returns MPCGS_OK (0) or a negative
+ *    code; no C++ exception crosses the ABI.  mpcgs_last_error() describes it.
+ *  - Pointers documented "host" are plain host memory owned by the caller,
+ *    read or written only during the call.  "device" pointers are CUDA global
+ *    memory on the context's device.
+ *  - Device memory is the caller's workspace (mpcgs_config.workspace) or, if
+ *    that is NULL, memory the context allocates and frees itself.
+ *  - MPCGS_E_CUDA and MPCGS_E_NCCL are sticky: after them only mpcgs_free()
+ *    and mpcgs_last_error() are valid on that context.
+ *  - A context is used by one host thread at a time.  Multi-GPU = one process
+ *    (one context) per GPU, ranks given in mpcgs_config.
+ *  - Tree arrays: 2n-1 nodes, tips 0..n-1 at age 0, interior nodes n..2n-2,
+ *    parent[root] = -1, age[] in mutation units (S22).
+ *  - Functions marked [host-only] never touch a GPU and work without one.
+ */
+#ifndef MPCGS_H
+#define MPCGS_H
+
+#include <stddef.h>
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+#define MPCGS_MAX_SEQ 1024        /* n <= 1024: node ids fit 11 bits, register need <= 10 */
+#define MPCGS_MAX_PROPOSALS 4096  /* N per step */
+#define MPCGS_MAX_GRID 4096       /* theta grid points */
+
+typedef struct mpcgs_ctx mpcgs_ctx;
+
+typedef enum {
+    MPCGS_OK = 0,
+    MPCGS_E_ARG = -1,        /* bad argument: n<3, L<1, theta0<=0, N<1, N%world!=0, capacity */
+    MPCGS_E_ALIGNMENT = -2,  /* a character outside ACGTacgt (S2) or unreadable PHYLIP */
+    MPCGS_E_STATE = -3,      /* call out of order (e.g. estimate before sample) */
+    MPCGS_E_CUDA = -4,       /* CUDA runtime error (sticky) */
+    MPCGS_E_NCCL = -5,       /* NCCL error or NCCL unavailable for world > 1 (sticky) */
+    MPCGS_E_NOMEM = -6,      /* workspace too small / allocation failed */
+    MPCGS_E_NUMERIC = -7     /* all N+1 weights non-finite (S6) */
+} mpcgs_status;
+
+/* Alignment D (5.1.1 L1229-1241): n rows of L characters in {A,C,G,T,a,c,g,t}.
+ * rows: host array of n pointers to L chars each; copied during mpcgs_init. */
+typedef struct {
+    int32_t n_seq;
+    int32_t n_sites;
+    const char* const* rows;
+} mpcgs_alignment;
+
+typedef struct {
+    double base_freq[4];   /* pi (Eq. 20); any entry < 0 -> empirical frequencies over all n*L
+                              characters (L702-703, S1) */
+    double mu;             /* F81 rate u; <= 0 -> 1/(1 - sum pi^2) (S3), 1 if sum pi^2 == 1 */
+    int32_t precision;     /* 64: FP64 partials (parity build) | 32: FP32 partials (fast) */
+    int32_t burnin_steps;  /* GMH steps before sampling; 1 draw each, not stored (Fig. 12, S17) */
+    int32_t max_proposals; /* capacity: largest N passed to mpcgs_sample (<= MPCGS_MAX_PROPOSALS) */
+    int64_t max_samples;   /* capacity: largest M passed to mpcgs_sample */
+    const int32_t* init_parent; /* host [2n-1] initial genealogy G0; NULL -> UPGMA (5.1.3, S19) */
+    const double* init_age;     /* host [2n-1]; used with init_parent */
+    int32_t rank, world;   /* world = 1: one GPU.  world > 1: proposals sharded over ranks */
+    const void* nccl_id;   /* host, 128 bytes: ncclUniqueId made by rank 0 with
+                              mpcgs_nccl_unique_id() and broadcast by the caller; NULL if world = 1 */
+    void* stream;          /* cudaStream_t for all work; NULL = the legacy default stream */
+    void* workspace;       /* device memory of >= mpcgs_workspace_bytes(...) bytes, 256-B aligned;
+                              NULL -> the context allocates (and frees) its own */
+    size_t workspace_bytes;
+} mpcgs_config;
+
+/* [host-only] Fill cfg with defaults: empirical pi, default u, precision 64, burn-in 0,
+ * max_proposals 1024, max_samples 1<<20, world 1. */
+void mpcgs_config_default(mpcgs_config* cfg);
+
+/* [host-only] Device bytes a context needs for these capacities. */
+size_t mpcgs_workspace_bytes(int32_t n_seq, int32_t n_sites, int32_t max_proposals,
+                             int64_t max_samples, int32_t precision);
+
+/* Create a context: validate and copy the alignment, compute pi and u, build G0
+ * (init_parent/init_age, else UPGMA), upload everything to the device and score
+ * P(D|G0) with the pruning kernel.  theta0 > 0 is the driving value (L1239-1241). */
+mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, double theta0,
+                        mpcgs_ctx** out);
+
+/* Same, reading a sequential PHYLIP file (5.1.1 L1233-1237): first line "n L", then
+ * per row a name (first 10 characters, or up to the first blank) and L bases. */
+mpcgs_status mpcgs_init_phylip(const char* path, const mpcgs_config* cfg, double theta0,
+                               mpcgs_ctx** out);
+
+/* Run burn-in then ceil(n_samples / n_proposals) sampling steps with N = n_proposals
+ * proposals per step (Alg. 1; Fig. 11/12).  Every random number is Philox4x32-10
+ * keyed by `seed` (S21), so results are identical for every world size (P22).
+ * Previous samples are discarded.  No host synchronisation inside the loop;
+ * returns after the work is complete. */
+mpcgs_status mpcgs_sample(mpcgs_ctx* ctx, int32_t n_proposals, int64_t n_samples, uint64_t seed);
+
+/* theta-hat = argmax L(theta) over the stored samples (Eq. 25-26; S20): a log-spaced
+ * grid of n_grid points (3..MPCGS_MAX_GRID) over [S_min, S_max]/(n-1) evaluated on
+ * the device, then safeguarded Newton on d lnL/d theta inside the best bracket.
+ * grid_theta / grid_logL: host [n_grid] or NULL; grid_logL = ln L(theta). */
+mpcgs_status mpcgs_estimate_theta(mpcgs_ctx* ctx, double* theta_hat, int32_t n_grid,
+                                  double* grid_theta, double* grid_logL);
+
+/* ln L(theta) (Eq. 25-26) of the stored samples at one theta (device reduction). */
+mpcgs_status mpcgs_log_rel_likelihood(mpcgs_ctx* ctx, double theta, double* out);
+
+/* Score arbitrary genealogies with the pruning kernel (Eq. 19-22): host parent/age
+ * [n_trees][2n-1] -> host logL_out [n_trees] (ln P(D|G)). */
+mpcgs_status mpcgs_score_trees(mpcgs_ctx* ctx, int32_t n_trees, const int32_t* parent,
+                               const double* age, double* logL_out);
+
+/* Replace the chain state (generator) by a host tree; its logL is recomputed. */
+mpcgs_status mpcgs_set_state(mpcgs_ctx* ctx, const int32_t* parent, const double* age);
+
+/* Read the generator: host parent/age [2n-1]; logL and S (nullable). */
+mpcgs_status mpcgs_get_state(mpcgs_ctx* ctx, int32_t* parent, double* age, double* logL,
+                             double* S);
+
+/* One GMH step at explicit step index `step` with N proposals and K draws (K <= N),
+ * the generator advancing to the last draw; nothing is stored in the sample store.
+ * Outputs (host, nullable): target node; per slot 0..N: logL[N+1], S[N+1],
+ * t12[(N+1)*2] (new ages of the target and parent ids; slot 0 = generator's),
+ * pair[N+1] (0:(c1,c2) 1:(c1,c3) 2:(c2,c3); -1 for slot 0); draws[K]. */
+mpcgs_status mpcgs_step_trace(mpcgs_ctx* ctx, int64_t step, int32_t n_proposals, int32_t n_draws,
+                              uint64_t seed, int32_t* target, double* logL, double* S,
+                              double* t12, int32_t* pair, int32_t* draws);
+
+/* Split GMH step for proposal sharding (S.8(e)): mpcgs_step_local computes this
+ * rank's proposal records (slots mpcgs_shard_range) for step `step`;
+ * mpcgs_get_records / mpcgs_put_records move records (5 doubles per slot:
+ * logL, S, t1, t2, pair) of slots [first, first+count) to / from host memory;
+ * mpcgs_step_finish draws K samples from all N+1 records and advances the
+ * generator.  With NCCL (world > 1) mpcgs_sample does the exchange itself. */
+mpcgs_status mpcgs_step_local(mpcgs_ctx* ctx, int64_t step, int32_t n_proposals, uint64_t seed);
+mpcgs_status mpcgs_get_records(mpcgs_ctx* ctx, int32_t first, int32_t count, double* host_rec);
+mpcgs_status mpcgs_put_records(mpcgs_ctx* ctx, int32_t first, int32_t count,
+                               const double* host_rec);
+mpcgs_status mpcgs_step_finish(mpcgs_ctx* ctx, int64_t step, int32_t n_proposals,
+                               int32_t n_draws, uint64_t seed, int32_t* draws);
+
+/* Copy samples [first, first+count) to host arrays (each nullable): coalescent
+ * statistic S_G = sum k(k-1)T_k (Eq. 18), ln P(D|G), step index, slot index. */
+mpcgs_status mpcgs_get_samples(mpcgs_ctx* ctx, int64_t first, int64_t count, double* S,
+                               double* logL, int64_t* step, int32_t* slot);
+int64_t mpcgs_num_samples(const mpcgs_ctx* ctx);
+
+/* Re-drive: theta0 <- theta (L791-797).  Cached P(D|G) stays valid (Eq. 23). */
+mpcgs_status mpcgs_set_theta0(mpcgs_ctx* ctx, double theta0);
+
+/* Model parameters actually used (host out: pi[4], u). */
+mpcgs_status mpcgs_get_model(const mpcgs_ctx* ctx, double* pi, double* mu);
+
+/* Timing mode for mpcgs_sample: on -> CUDA events bracket every pruning launch
+ * (and the loop runs as plain launches, not a CUDA graph). */
+mpcgs_status mpcgs_set_timing(mpcgs_ctx* ctx, int32_t on);
+
+/* Device time (ms) of the last mpcgs_sample loop and of its pruning launches
+ * (CUDA events on the context stream), and kernel launches it issued. */
+mpcgs_status mpcgs_last_timing(const mpcgs_ctx* ctx, double* loop_ms, double* prune_ms,
+                               int64_t* launches);
+
+const char* mpcgs_last_error(const mpcgs_ctx* ctx);
+void mpcgs_free(mpcgs_ctx* ctx);
+
+/* ---------------------------------------------------------------- host-only helpers */
+/* [host-only] Proposal slots owned by `rank`: slots first..first+count-1 of 1..N. */
+mpcgs_status mpcgs_shard_range(int32_t n_proposals, int32_t rank, int32_t world, int32_t* first,
+                               int32_t* count);
+/* [host-only] UPGMA G0 (5.1.3 L1287-1295, S19) from codes[n][L] in {0..3}. */
+mpcgs_status mpcgs_upgma(int32_t n_seq, int32_t n_sites, const uint8_t* codes, double theta0,
+                         int32_t* parent, double* age);
+/* [host-only] Post-order register schedule of a tree as used by the pruning kernel
+ * (DESIGN.md "prune"): op[i] = type | sp<<2 | tipA<<6 | tipB<<17, e[2i], e[2i+1] branch
+ * factors exp(-u t); returns the register need (max stack depth) or < 0 on error. */
+int32_t mpcgs_tree_schedule(int32_t n_seq, const int32_t* parent, const double* age, double mu,
+                            uint32_t* op, double* e);
+/* [host-only] Sequential PHYLIP reader: dims, then rows (n*L chars, row-major). */
+mpcgs_status mpcgs_phylip_dims(const char* path, int32_t* n_seq, int32_t* n_sites);
+mpcgs_status mpcgs_phylip_read(const char* path, char* seqs, int32_t cap_chars);
+/* [host-only] Philox4x32-10 block (for known-answer checks of the device generator). */
+void mpcgs_philox(const uint32_t ctr[4], const uint32_t key[2], uint32_t out[4]);
+/* [host-only] A fresh ncclUniqueId (128 bytes) via the dynamically loaded NCCL. */
+mpcgs_status mpcgs_nccl_unique_id(void* out128);
+const char* mpcgs_version(void);
+
+#ifdef __cplusplus
+}
+#endif
+#endif

@@ -1,0 +1,1072 @@
+// host.cu -- the C ABI (include/mpcgs.h): validation, model setup, G0, device
+// workspace layout, the device-resident step loop, theta estimation, NCCL.
+//
+// Host code here never computes the method's hot path: every per-step
+// quantity (targets, contexts, proposals, likelihoods, weights, draws, theta
+// curve) is computed by the kernels in step.cu / prune.cu / theta.cu.  The host
+// builds G0 (UPGMA, 5.1.3 L1287-1295) and the post-order schedule of trees it
+// is handed (mpcgs_score_trees / set_state), and drives Newton on the theta
+// bracket with device reductions.
+#include <dlfcn.h>
+#include <nccl.h>
+
+#include <algorithm>
+#include <cmath>
+#include <cstdio>
+#include <cstdlib>
+#include <cstring>
+#include <string>
+#include <vector>
+
+#include "common.cuh"
+#include "kernels.cuh"
+#include "mpcgs.h"
+
+using namespace mpcgs;
+
+// ---------------------------------------------------------------- NCCL (dlopen)
+namespace {
+struct NcclApi {
+    bool ok = false;
+    ncclResult_t (*getUniqueId)(ncclUniqueId*) = nullptr;
+    ncclResult_t (*commInitRank)(ncclComm_t*, int, ncclUniqueId, int) = nullptr;
+    ncclResult_t (*allGather)(const void*, void*, size_t, ncclDataType_t, ncclComm_t, cudaStream_t) = nullptr;
+    ncclResult_t (*commDestroy)(ncclComm_t) = nullptr;
+    const char* (*errStr)(ncclResult_t) = nullptr;
+};
+NcclApi& nccl() {
+    static NcclApi api;
+    static bool tried = false;
+    if (!tried) {
+        tried = true;
+        void* h = dlopen("libnccl.so.2", RTLD_NOW | RTLD_GLOBAL);
+        if (!h) h = dlopen("libnccl.so", RTLD_NOW | RTLD_GLOBAL);
+        if (h) {
+            api.getUniqueId = (decltype(api.getUniqueId))dlsym(h, "ncclGetUniqueId");
+            api.commInitRank = (decltype(api.commInitRank))dlsym(h, "ncclCommInitRank");
+            api.allGather = (decltype(api.allGather))dlsym(h, "ncclAllGather");
+            api.commDestroy = (decltype(api.commDestroy))dlsym(h, "ncclCommDestroy");
+            api.errStr = (decltype(api.errStr))dlsym(h, "ncclGetErrorString");
+            api.ok = api.getUniqueId && api.commInitRank && api.allGather && api.commDestroy;
+        }
+    }
+    return api;
+}
+}  // namespace
+
+// ---------------------------------------------------------------- context
+struct mpcgs_ctx {
+    DevState s{};
+    int n = 0, L = 0, nn = 0, Lpad = 0, nops = 0, depth = 0, precision = 64;
+    int world = 1, rank = 0, burnin = 0;
+    int Nmax = 0;
+    int64_t Mmax = 0;
+    double theta0 = 0.0, sample_theta0 = 0.0;
+    cudaStream_t user = nullptr, work = nullptr;
+    void* ws = nullptr;
+    size_t ws_bytes = 0;
+    bool own_ws = false;
+    double* score_out = nullptr;
+    unsigned* theta_cnt = nullptr;
+    int64_t nsamples = 0;
+    int lastN = 0;
+    bool sticky = false;
+    std::string err;
+    ncclComm_t comm = nullptr;
+    bool timing = false;
+    double loop_ms = 0.0, prune_ms = 0.0;
+    int64_t launches = 0;
+    std::vector<cudaEvent_t> evpool;
+    cudaEvent_t ev_a = nullptr, ev_b = nullptr;
+    std::vector<double> pinned_dummy;
+};
+
+namespace {
+
+mpcgs_status fail(mpcgs_ctx* c, mpcgs_status st, const std::string& msg) {
+    if (c) {
+        c->err = msg;
+        if (st == MPCGS_E_CUDA || st == MPCGS_E_NCCL) c->sticky = true;
+    }
+    return st;
+}
+
+#define CU(call)                                                                                  \
+    do {                                                                                          \
+        cudaError_t e_ = (call);                                                                  \
+        if (e_ != cudaSuccess)                                                                    \
+            return fail(c, MPCGS_E_CUDA, std::string(#call) + ": " + cudaGetErrorString(e_));      \
+    } while (0)
+
+#define CHECK_CTX(c)                                                               \
+    do {                                                                           \
+        if (!(c)) return MPCGS_E_ARG;                                              \
+        if ((c)->sticky) return MPCGS_E_CUDA;                                      \
+    } while (0)
+
+// ------------------------------------------------------------ workspace layout
+struct Layout {
+    size_t codes, parent, left, right, need, age, e, em, gen, ctx_i, ctx_d, tau, len, lcnt, entry, omega, fixed;
+    size_t rec, sched_op, sched_e, tile_part, tile_cnt, sS, sL, sStep, sSlot, counters, last_draws, theta_buf,
+        theta_cnt, score_out, total;
+    int tiles_max;
+};
+
+size_t al(size_t x) { return (x + 255) & ~(size_t)255; }
+
+Layout layout(int n, int L, int Nmax, int64_t Mmax, int precision) {
+    Layout y{};
+    const int nn = 2 * n - 1, nops = n - 1;
+    const int Lpad = (L + 15) & ~15;
+    const size_t esz = precision == 32 ? sizeof(float4) : sizeof(double4);
+    y.tiles_max = (L + PRUNE_THREADS - 1) / PRUNE_THREADS;
+    size_t o = 0;
+    auto take = [&](size_t bytes) {
+        size_t r = o;
+        o += al(bytes);
+        return r;
+    };
+    y.codes = take((size_t)n * Lpad);
+    y.parent = take(4 * (size_t)nn);
+    y.left = take(4 * (size_t)nn);
+    y.right = take(4 * (size_t)nn);
+    y.need = take(4 * (size_t)nn);
+    y.age = take(8 * (size_t)nn);
+    y.e = take(8 * (size_t)nn);
+    y.em = take(8 * (size_t)nn);
+    y.gen = take(8 * 4);
+    y.ctx_i = take(4 * 16);
+    y.ctx_d = take(8 * 8);
+    y.tau = take(8 * (size_t)(n + 2));
+    y.len = take(8 * (size_t)(n + 1));
+    y.lcnt = take(4 * (size_t)(n + 1));
+    y.entry = take(4 * (size_t)(n + 2));
+    y.omega = take(8 * 9 * (size_t)(n + 1));
+    y.fixed = take(8 * (size_t)n);
+    y.rec = take(8 * REC * (size_t)(Nmax + 1));
+    y.sched_op = take(4 * (size_t)Nmax * nops);
+    y.sched_e = take(esz * (size_t)Nmax * nops);
+    y.tile_part = take(8 * (size_t)Nmax * y.tiles_max);
+    y.tile_cnt = take(4 * (size_t)Nmax);
+    y.sS = take(8 * (size_t)std::max<int64_t>(Mmax, 1));
+    y.sL = take(8 * (size_t)std::max<int64_t>(Mmax, 1));
+    y.sStep = take(8 * (size_t)std::max<int64_t>(Mmax, 1));
+    y.sSlot = take(4 * (size_t)std::max<int64_t>(Mmax, 1));
+    y.counters = take(8 * 8);
+    y.last_draws = take(4 * (size_t)Nmax);
+    y.theta_buf = take(8 * (size_t)(2 * MPCGS_MAX_GRID + 3 * 296 + 16));
+    y.theta_cnt = take(16);
+    y.score_out = take(8 * (size_t)Nmax);
+    y.total = o;
+    return y;
+}
+
+// ------------------------------------------------------------ host tree helpers
+int check_tree(int n, const int32_t* parent, const double* age, std::string& why) {
+    const int nn = 2 * n - 1;
+    std::vector<int> kids(nn, 0);
+    int roots = 0;
+    for (int v = 0; v < nn; ++v) {
+        const int p = parent[v];
+        if (p < 0) {
+            ++roots;
+            if (v < n) { why = "a tip has no parent"; return -1; }
+            continue;
+        }
+        if (p < n || p >= nn) { why = "parent id out of the interior range"; return -1; }
+        if (!(age[p] >= age[v])) { why = "a parent is younger than its child"; return -1; }
+        if (!std::isfinite(age[v])) { why = "non-finite age"; return -1; }
+        ++kids[p];
+    }
+    if (roots != 1) { why = "tree must have exactly one root"; return -1; }
+    for (int v = 0; v < n; ++v)
+        if (age[v] != 0.0) { why = "tips must have age 0 (S22)"; return -1; }
+    for (int v = n; v < nn; ++v)
+        if (kids[v] != 2) { why = "interior nodes need two children"; return -1; }
+    // acyclic: every node reaches the root in < nn steps
+    for (int v = 0; v < nn; ++v) {
+        int x = v, k = 0;
+        while (parent[x] >= 0 && k < nn) { x = parent[x]; ++k; }
+        if (k >= nn) { why = "cycle in parent array"; return -1; }
+    }
+    return 0;
+}
+
+struct HostTree {
+    std::vector<int32_t> left, right, need;
+    std::vector<double> e, em;
+    int root = -1;
+};
+
+// children (lower id first), Sethi-Ullman needs (post-order), branch factors
+void host_tree(int n, const int32_t* parent, const double* age, double u, HostTree& t) {
+    const int nn = 2 * n - 1;
+    t.left.assign(nn, -1);
+    t.right.assign(nn, -1);
+    t.need.assign(nn, 0);
+    t.e.assign(nn, 1.0);
+    t.em.assign(nn, 0.0);
+    for (int v = 0; v < nn; ++v) {
+        const int p = parent[v];
+        if (p < 0) { t.root = v; continue; }
+        if (t.left[p] < 0) t.left[p] = v;
+        else if (v < t.left[p]) { t.right[p] = t.left[p]; t.left[p] = v; }
+        else t.right[p] = v;
+        const double len = age[p] - age[v];
+        t.e[v] = std::exp(-u * len);
+        t.em[v] = -std::expm1(-u * len);
+    }
+    // post-order by an explicit stack
+    std::vector<int> st;
+    std::vector<char> done(nn, 0);
+    st.push_back(t.root);
+    while (!st.empty()) {
+        int v = st.back();
+        if (v < n) { st.pop_back(); continue; }
+        const int a = t.left[v], b = t.right[v];
+        if ((a >= n && !done[a]) || (b >= n && !done[b])) {
+            if (a >= n && !done[a]) st.push_back(a);
+            if (b >= n && !done[b]) st.push_back(b);
+            continue;
+        }
+        t.need[v] = su_need(a < n ? 0 : t.need[a], b < n ? 0 : t.need[b]);
+        done[v] = 1;
+        st.pop_back();
+    }
+}
+
+template <typename ET>
+int host_schedule(int n, const HostTree& t, uint32_t* op, ET* e4) {
+    std::vector<int> stack(2 * n + 4);
+    return emit_schedule(
+        n, t.root, [&](int v) { return t.left[v]; }, [&](int v) { return t.right[v]; },
+        [&](int v) { return v < n ? 0 : t.need[v]; },
+        [&](int i, uint32_t code, int ca, int cb) {
+            op[i] = code;
+            e4[4 * i + 0] = (ET)t.e[ca];
+            e4[4 * i + 1] = (ET)t.em[ca];
+            e4[4 * i + 2] = (ET)t.e[cb];
+            e4[4 * i + 3] = (ET)t.em[cb];
+        },
+        stack.data());
+}
+
+double host_S(int n, const double* age) {
+    // S = sum_k k(k-1) T_k = 2 sum_i (n-i) h_i over sorted coalescence ages (Eq. 18)
+    std::vector<double> h(age + n, age + 2 * n - 1);
+    std::sort(h.begin(), h.end());
+    double S = 0.0;
+    for (int i = 1; i <= n - 1; ++i) S += 2.0 * (double)(n - i) * h[i - 1];
+    return S;
+}
+
+int code_of(char ch) {
+    switch (ch) {
+        case 'A': case 'a': return 0;
+        case 'C': case 'c': return 1;
+        case 'G': case 'g': return 2;
+        case 'T': case 't': return 3;
+        default: return -1;
+    }
+}
+
+// UPGMA (5.1.3 L1287-1295): Hamming distances, average linkage over leaf pairs,
+// node height theta0 * d / 2 forced 1e-6 theta0 above the children (S19).
+void upgma(int n, int L, const uint8_t* codes, double theta0, int32_t* parent, double* age) {
+    const int nn = 2 * n - 1;
+    std::vector<std::vector<double>> d(nn, std::vector<double>(nn, 0.0));
+    for (int i = 0; i < n; ++i)
+        for (int j = i + 1; j < n; ++j) {
+            long diff = 0;
+            const uint8_t* a = codes + (size_t)i * L;
+            const uint8_t* b = codes + (size_t)j * L;
+            for (int s = 0; s < L; ++s) diff += a[s] != b[s];
+            d[i][j] = d[j][i] = (double)diff;
+        }
+    std::vector<int> live(n), size(nn, 1);
+    for (int i = 0; i < n; ++i) live[i] = i;
+    for (int v = 0; v < nn; ++v) { parent[v] = -1; age[v] = 0.0; }
+    for (int k = n; k < nn; ++k) {
+        // closest pair; ties -> smallest (lower id, higher id) in lexicographic order
+        int bi = -1, bj = -1;
+        double best = 0.0;
+        for (size_t x = 0; x < live.size(); ++x)
+            for (size_t y = x + 1; y < live.size(); ++y) {
+                int i = std::min(live[x], live[y]), j = std::max(live[x], live[y]);
+                double dv = d[i][j];
+                if (bi < 0 || dv < best || (dv == best && (i < bi || (i == bi && j < bj)))) {
+                    best = dv; bi = i; bj = j;
+                }
+            }
+        double h = theta0 * best / 2.0;
+        h = std::max(h, std::max(age[bi], age[bj]) + 1e-6 * theta0);
+        age[k] = h;
+        parent[bi] = parent[bj] = k;
+        size[k] = size[bi] + size[bj];
+        std::vector<int> next;
+        for (int v : live)
+            if (v != bi && v != bj) next.push_back(v);
+        for (int v : next) {
+            double dv = (size[bi] * d[bi][v] + size[bj] * d[bj][v]) / (double)size[k];
+            d[k][v] = d[v][k] = dv;
+        }
+        next.push_back(k);
+        live.swap(next);
+    }
+}
+
+// sites per CTA so that the pruning grid has enough CTAs (>= ~8 per SM)
+void prune_tiling(int L, int ntrees, int& tiles, int& sites_per_cta) {
+    long want = (long)148 * 8;
+    int spt = (int)std::max<long>(1, std::min<long>(16, ((long)ntrees * L) / (PRUNE_THREADS * want)));
+    sites_per_cta = spt * PRUNE_THREADS;
+    tiles = (L + sites_per_cta - 1) / sites_per_cta;
+}
+
+PruneArgs prune_args(mpcgs_ctx* c, int ntrees, double* out, int out_first, int out_stride) {
+    PruneArgs a{};
+    a.codes = c->s.codes;
+    a.Lpad = c->Lpad;
+    a.L = c->L;
+    a.nops = c->nops;
+    for (int i = 0; i < 4; ++i) a.pi[i] = c->s.pi[i];
+    a.sched_op = c->s.sched_op;
+    a.sched_e = c->s.sched_e;
+    prune_tiling(c->L, ntrees, a.tiles, a.sites_per_cta);
+    a.tile_part = c->s.tile_part;
+    a.tile_cnt = c->s.tile_cnt;
+    a.out = out;
+    a.out_first = out_first;
+    a.out_stride = out_stride;
+    return a;
+}
+
+// enter / leave: order work on the internal stream after the user's stream
+mpcgs_status enter(mpcgs_ctx* c) {
+    CU(cudaEventRecord(c->ev_a, c->user));
+    CU(cudaStreamWaitEvent(c->work, c->ev_a, 0));
+    return MPCGS_OK;
+}
+mpcgs_status leave(mpcgs_ctx* c) {
+    CU(cudaStreamSynchronize(c->work));
+    return MPCGS_OK;
+}
+
+// upload schedules of host trees [first, first+count) and score them into score_out
+mpcgs_status score_batch(mpcgs_ctx* c, int count, const int32_t* parent, const double* age, double* out) {
+    const int n = c->n, nn = c->nn, nops = c->nops;
+    std::vector<uint32_t> ops((size_t)count * nops);
+    std::vector<double> e8;
+    std::vector<float> e4;
+    if (c->precision == 32) e4.resize((size_t)count * nops * 4);
+    else e8.resize((size_t)count * nops * 4);
+    for (int t = 0; t < count; ++t) {
+        std::string why;
+        if (check_tree(n, parent + (size_t)t * nn, age + (size_t)t * nn, why))
+            return fail(c, MPCGS_E_ARG, "tree " + std::to_string(t) + ": " + why);
+        HostTree ht;
+        host_tree(n, parent + (size_t)t * nn, age + (size_t)t * nn, c->s.u, ht);
+        int d = c->precision == 32 ? host_schedule<float>(n, ht, ops.data() + (size_t)t * nops,
+                                                          e4.data() + (size_t)t * nops * 4)
+                                   : host_schedule<double>(n, ht, ops.data() + (size_t)t * nops,
+                                                           e8.data() + (size_t)t * nops * 4);
+        if (d > c->depth) return fail(c, MPCGS_E_ARG, "tree needs more registers than compiled");
+    }
+    CU(cudaMemcpyAsync(c->s.sched_op, ops.data(), ops.size() * 4, cudaMemcpyHostToDevice, c->work));
+    if (c->precision == 32)
+        CU(cudaMemcpyAsync(c->s.sched_e, e4.data(), e4.size() * 4, cudaMemcpyHostToDevice, c->work));
+    else
+        CU(cudaMemcpyAsync(c->s.sched_e, e8.data(), e8.size() * 8, cudaMemcpyHostToDevice, c->work));
+    PruneArgs a = prune_args(c, count, c->score_out, 0, 1);
+    CU(launch_prune(a, count, c->depth, c->precision, c->work));
+    CU(cudaMemcpyAsync(out, c->score_out, 8 * (size_t)count, cudaMemcpyDeviceToHost, c->work));
+    CU(cudaStreamSynchronize(c->work));
+    return MPCGS_OK;
+}
+
+mpcgs_status upload_state(mpcgs_ctx* c, const int32_t* parent, const double* age) {
+    const int n = c->n, nn = c->nn;
+    std::string why;
+    if (check_tree(n, parent, age, why)) return fail(c, MPCGS_E_ARG, "generator: " + why);
+    HostTree ht;
+    host_tree(n, parent, age, c->s.u, ht);
+    if (ht.need[ht.root] > c->depth) return fail(c, MPCGS_E_ARG, "tree needs more registers than compiled");
+    double logL = 0.0;
+    mpcgs_status st = score_batch(c, 1, parent, age, &logL);
+    if (st) return st;
+    double gen[2] = {logL, host_S(n, age)};
+    CU(cudaMemcpyAsync(c->s.parent, parent, 4 * (size_t)nn, cudaMemcpyHostToDevice, c->work));
+    CU(cudaMemcpyAsync(c->s.left, ht.left.data(), 4 * (size_t)nn, cudaMemcpyHostToDevice, c->work));
+    CU(cudaMemcpyAsync(c->s.right, ht.right.data(), 4 * (size_t)nn, cudaMemcpyHostToDevice, c->work));
+    CU(cudaMemcpyAsync(c->s.need, ht.need.data(), 4 * (size_t)nn, cudaMemcpyHostToDevice, c->work));
+    CU(cudaMemcpyAsync(c->s.age, age, 8 * (size_t)nn, cudaMemcpyHostToDevice, c->work));
+    CU(cudaMemcpyAsync(c->s.e, ht.e.data(), 8 * (size_t)nn, cudaMemcpyHostToDevice, c->work));
+    CU(cudaMemcpyAsync(c->s.em, ht.em.data(), 8 * (size_t)nn, cudaMemcpyHostToDevice, c->work));
+    CU(cudaMemcpyAsync(c->s.gen, gen, 16, cudaMemcpyHostToDevice, c->work));
+    CU(cudaStreamSynchronize(c->work));
+    return MPCGS_OK;
+}
+
+mpcgs_status check_status(mpcgs_ctx* c) {
+    int64_t st = 0;
+    CU(cudaMemcpy(&st, c->s.counters + 2, 8, cudaMemcpyDeviceToHost));
+    if (st & STATUS_NUMERIC) return fail(c, MPCGS_E_NUMERIC, "all N+1 weights are non-finite");
+    if (st & STATUS_WALK) return fail(c, MPCGS_E_NUMERIC, "resimulation walk did not reach the ancestor");
+    return MPCGS_OK;
+}
+
+// one step's proposal work for this rank: context, propose, prune
+mpcgs_status step_local_launch(mpcgs_ctx* c, uint64_t seed, int64_t step, int N, bool timed, int ev_idx) {
+    int first = 1 + c->rank * (N / c->world), count = N / c->world;
+    CU(launch_context(c->s, seed, step, c->work));
+    CU(launch_propose(c->s, seed, step, first, count, c->work));
+    PruneArgs a = prune_args(c, count, c->s.rec, first, REC);
+    if (timed) CU(cudaEventRecord(c->evpool[2 * ev_idx], c->work));
+    CU(launch_prune(a, count, c->depth, c->precision, c->work));
+    if (timed) CU(cudaEventRecord(c->evpool[2 * ev_idx + 1], c->work));
+    c->launches += 3;
+    return MPCGS_OK;
+}
+
+mpcgs_status allgather_records(mpcgs_ctx* c, int N) {
+    if (c->world == 1) return MPCGS_OK;
+    NcclApi& api = nccl();
+    const size_t cnt = (size_t)(N / c->world) * REC;
+    double* recv = c->s.rec + REC;  // slot 1
+    ncclResult_t r = api.allGather(recv + c->rank * cnt, recv, cnt, ncclFloat64, c->comm, c->work);
+    if (r != ncclSuccess) return fail(c, MPCGS_E_NCCL, std::string("ncclAllGather: ") + (api.errStr ? api.errStr(r) : "?"));
+    return MPCGS_OK;
+}
+
+}  // namespace
+
+// ======================================================================== ABI
+extern "C" {
+
+const char* mpcgs_version(void) { return "mpcgs-b200 0.1 (sm_100a)"; }
+
+void mpcgs_config_default(mpcgs_config* cfg) {
+    if (!cfg) return;
+    std::memset(cfg, 0, sizeof(*cfg));
+    for (int i = 0; i < 4; ++i) cfg->base_freq[i] = -1.0;
+    cfg->mu = 0.0;
+    cfg->precision = 64;
+    cfg->burnin_steps = 0;
+    cfg->max_proposals = 1024;
+    cfg->max_samples = 1 << 20;
+    cfg->rank = 0;
+    cfg->world = 1;
+}
+
+size_t mpcgs_workspace_bytes(int32_t n_seq, int32_t n_sites, int32_t max_proposals, int64_t max_samples,
+                             int32_t precision) {
+    if (n_seq < 2 || n_sites < 1 || max_proposals < 1 || max_samples < 0) return 0;
+    return layout(n_seq, n_sites, max_proposals, max_samples, precision).total;
+}
+
+void mpcgs_philox(const uint32_t ctr[4], const uint32_t key[2], uint32_t out[4]) {
+    U4 r = philox(U4{ctr[0], ctr[1], ctr[2], ctr[3]}, key[0], key[1]);
+    out[0] = r.x;
+    out[1] = r.y;
+    out[2] = r.z;
+    out[3] = r.w;
+}
+
+mpcgs_status mpcgs_shard_range(int32_t N, int32_t rank, int32_t world, int32_t* first, int32_t* count) {
+    if (N < 1 || world < 1 || rank < 0 || rank >= world || N % world != 0 || !first || !count) return MPCGS_E_ARG;
+    *count = N / world;
+    *first = 1 + rank * (*count);
+    return MPCGS_OK;
+}
+
+mpcgs_status mpcgs_upgma(int32_t n, int32_t L, const uint8_t* codes, double theta0, int32_t* parent, double* age) {
+    if (n < 2 || L < 0 || !codes || !parent || !age || !(theta0 > 0)) return MPCGS_E_ARG;
+    upgma(n, L, codes, theta0, parent, age);
+    return MPCGS_OK;
+}
+
+int32_t mpcgs_tree_schedule(int32_t n, const int32_t* parent, const double* age, double mu, uint32_t* op,
+                            double* e) {
+    if (n < 2 || n > MPCGS_MAX_SEQ || !parent || !age || !op || !e) return MPCGS_E_ARG;
+    std::string why;
+    if (check_tree(n, parent, age, why)) return MPCGS_E_ARG;
+    HostTree ht;
+    host_tree(n, parent, age, mu, ht);
+    return host_schedule<double>(n, ht, op, e);
+}
+
+mpcgs_status mpcgs_phylip_dims(const char* path, int32_t* n_seq, int32_t* n_sites) {
+    FILE* f = path ? std::fopen(path, "r") : nullptr;
+    if (!f) return MPCGS_E_ALIGNMENT;
+    int n = 0, L = 0;
+    int ok = std::fscanf(f, "%d %d", &n, &L);
+    std::fclose(f);
+    if (ok != 2 || n < 1 || L < 1) return MPCGS_E_ALIGNMENT;
+    *n_seq = n;
+    *n_sites = L;
+    return MPCGS_OK;
+}
+
+mpcgs_status mpcgs_phylip_read(const char* path, char* seqs, int32_t cap) {
+    int32_t n, L;
+    if (mpcgs_phylip_dims(path, &n, &L) != MPCGS_OK) return MPCGS_E_ALIGNMENT;
+    if ((int64_t)n * L > cap) return MPCGS_E_ARG;
+    FILE* f = std::fopen(path, "r");
+    if (!f) return MPCGS_E_ALIGNMENT;
+    std::vector<char> line(1 << 16);
+    std::string all;
+    {
+        int c;
+        std::string cur;
+        while ((c = std::fgetc(f)) != EOF) all.push_back((char)c);
+    }
+    std::fclose(f);
+    size_t pos = all.find('\n');
+    if (pos == std::string::npos) return MPCGS_E_ALIGNMENT;
+    ++pos;
+    for (int r = 0; r < n; ++r) {
+        // skip blank lines
+        while (pos < all.size() && (all[pos] == '\n' || all[pos] == '\r')) ++pos;
+        size_t eol = all.find('\n', pos);
+        if (eol == std::string::npos) eol = all.size();
+        std::string ln = all.substr(pos, eol - pos);
+        pos = eol + 1;
+        // name: first 10 characters, or up to the first blank inside them (S2)
+        size_t cut = std::min<size_t>(10, ln.size());
+        for (size_t i = 0; i < cut; ++i)
+            if (ln[i] == ' ' || ln[i] == '\t') { cut = i; break; }
+        std::string rest = ln.substr(cut);
+        int got = 0;
+        auto eat = [&](const std::string& s) {
+            for (char ch : s) {
+                if (ch == ' ' || ch == '\t' || ch == '\r') continue;
+                if (got >= L) return false;
+                if (code_of(ch) < 0) return false;
+                seqs[(size_t)r * L + got++] = ch;
+            }
+            return true;
+        };
+        if (!eat(rest)) return MPCGS_E_ALIGNMENT;
+        while (got < L && pos < all.size()) {  // wrapped sequential format
+            eol = all.find('\n', pos);
+            if (eol == std::string::npos) eol = all.size();
+            std::string more = all.substr(pos, eol - pos);
+            pos = eol + 1;
+            if (!eat(more)) return MPCGS_E_ALIGNMENT;
+        }
+        if (got != L) return MPCGS_E_ALIGNMENT;
+    }
+    return MPCGS_OK;
+}
+
+mpcgs_status mpcgs_nccl_unique_id(void* out128) {
+    NcclApi& api = nccl();
+    if (!api.ok || !out128) return MPCGS_E_NCCL;
+    ncclUniqueId id;
+    if (api.getUniqueId(&id) != ncclSuccess) return MPCGS_E_NCCL;
+    std::memcpy(out128, &id, sizeof(id));
+    return MPCGS_OK;
+}
+
+mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, double theta0, mpcgs_ctx** out) {
+    if (!out) return MPCGS_E_ARG;
+    *out = nullptr;
+    if (!aln || !cfg || !aln->rows) return MPCGS_E_ARG;
+    const int n = aln->n_seq, L = aln->n_sites;
+    if (n < 3 || n > MPCGS_MAX_SEQ || L < 1 || !(theta0 > 0.0) || !std::isfinite(theta0)) return MPCGS_E_ARG;
+    if (cfg->precision != 32 && cfg->precision != 64) return MPCGS_E_ARG;
+    if (cfg->max_proposals < 1 || cfg->max_proposals > MPCGS_MAX_PROPOSALS || cfg->max_samples < 0) return MPCGS_E_ARG;
+    if (cfg->world < 1 || cfg->rank < 0 || cfg->rank >= cfg->world || cfg->burnin_steps < 0) return MPCGS_E_ARG;
+    // alignment -> codes (S2: ACGT only)
+    std::vector<uint8_t> codes((size_t)n * L);
+    for (int i = 0; i < n; ++i) {
+        if (!aln->rows[i]) return MPCGS_E_ARG;
+        for (int s = 0; s < L; ++s) {
+            int cd = code_of(aln->rows[i][s]);
+            if (cd < 0) return MPCGS_E_ALIGNMENT;
+            codes[(size_t)i * L + s] = (uint8_t)cd;
+        }
+    }
+    mpcgs_ctx* c = new mpcgs_ctx();
+    c->n = n;
+    c->L = L;
+    c->nn = 2 * n - 1;
+    c->Lpad = (L + 15) & ~15;
+    c->nops = n - 1;
+    c->depth = prune_depth_for(n);
+    c->precision = cfg->precision;
+    c->world = cfg->world;
+    c->rank = cfg->rank;
+    c->burnin = cfg->burnin_steps;
+    c->Nmax = cfg->max_proposals;
+    c->Mmax = cfg->max_samples;
+    c->theta0 = theta0;
+    c->user = (cudaStream_t)cfg->stream;
+    // model (Eq. 20): pi empirical unless given (S1); u = 1/(1 - sum pi^2) unless given (S3)
+    double pi[4];
+    bool emp = false;
+    for (int i = 0; i < 4; ++i) emp |= cfg->base_freq[i] < 0.0;
+    if (emp) {
+        double cnt[4] = {0, 0, 0, 0};
+        for (uint8_t x : codes) cnt[x] += 1.0;
+        for (int i = 0; i < 4; ++i) pi[i] = cnt[i] / ((double)n * L);
+    } else {
+        double sum = 0.0;
+        for (int i = 0; i < 4; ++i) { pi[i] = cfg->base_freq[i]; sum += pi[i]; }
+        if (!(std::fabs(sum - 1.0) < 1e-9)) { delete c; return MPCGS_E_ARG; }
+    }
+    double sq = pi[0] * pi[0] + pi[1] * pi[1] + pi[2] * pi[2] + pi[3] * pi[3];
+    double u = cfg->mu > 0.0 ? cfg->mu : (sq < 1.0 ? 1.0 / (1.0 - sq) : 1.0);
+    // G0
+    std::vector<int32_t> parent(c->nn);
+    std::vector<double> age(c->nn);
+    if (cfg->init_parent && cfg->init_age) {
+        std::copy(cfg->init_parent, cfg->init_parent + c->nn, parent.begin());
+        std::copy(cfg->init_age, cfg->init_age + c->nn, age.begin());
+    } else {
+        upgma(n, L, codes.data(), theta0, parent.data(), age.data());
+    }
+    // device memory
+    Layout y = layout(n, L, c->Nmax, c->Mmax, c->precision);
+    mpcgs_status st = MPCGS_OK;
+    do {
+        if (cudaStreamCreateWithFlags(&c->work, cudaStreamNonBlocking) != cudaSuccess ||
+            cudaEventCreateWithFlags(&c->ev_a, cudaEventDisableTiming) != cudaSuccess ||
+            cudaEventCreate(&c->ev_b) != cudaSuccess) {
+            st = fail(c, MPCGS_E_CUDA, "stream/event creation failed (no CUDA device?)");
+            break;
+        }
+        if (cfg->workspace) {
+            if (cfg->workspace_bytes < y.total || ((uintptr_t)cfg->workspace & 255)) {
+                st = fail(c, MPCGS_E_NOMEM, "workspace too small or not 256-byte aligned");
+                break;
+            }
+            c->ws = cfg->workspace;
+            c->ws_bytes = cfg->workspace_bytes;
+        } else {
+            if (cudaMalloc(&c->ws, y.total) != cudaSuccess) {
+                st = fail(c, MPCGS_E_NOMEM, "cudaMalloc of the workspace failed");
+                break;
+            }
+            c->own_ws = true;
+            c->ws_bytes = y.total;
+        }
+        char* b = (char*)c->ws;
+        DevState& s = c->s;
+        s.n = n; s.nn = c->nn; s.L = L; s.Lpad = c->Lpad; s.nops = c->nops; s.precision = c->precision;
+        for (int i = 0; i < 4; ++i) s.pi[i] = pi[i];
+        s.u = u;
+        s.theta0 = theta0;
+        s.codes = (const uint8_t*)(b + y.codes);
+        s.parent = (int32_t*)(b + y.parent);
+        s.left = (int32_t*)(b + y.left);
+        s.right = (int32_t*)(b + y.right);
+        s.need = (int32_t*)(b + y.need);
+        s.age = (double*)(b + y.age);
+        s.e = (double*)(b + y.e);
+        s.em = (double*)(b + y.em);
+        s.gen = (double*)(b + y.gen);
+        s.ctx_i = (int32_t*)(b + y.ctx_i);
+        s.ctx_d = (double*)(b + y.ctx_d);
+        s.tau = (double*)(b + y.tau);
+        s.len = (double*)(b + y.len);
+        s.lcnt = (int32_t*)(b + y.lcnt);
+        s.entry = (int32_t*)(b + y.entry);
+        s.omega = (double*)(b + y.omega);
+        s.fixed = (double*)(b + y.fixed);
+        s.rec = (double*)(b + y.rec);
+        s.sched_op = (uint32_t*)(b + y.sched_op);
+        s.sched_e = (void*)(b + y.sched_e);
+        s.tile_part = (double*)(b + y.tile_part);
+        s.tile_cnt = (uint32_t*)(b + y.tile_cnt);
+        s.sS = (double*)(b + y.sS);
+        s.sL = (double*)(b + y.sL);
+        s.sStep = (int64_t*)(b + y.sStep);
+        s.sSlot = (int32_t*)(b + y.sSlot);
+        s.counters = (int64_t*)(b + y.counters);
+        s.last_draws = (int32_t*)(b + y.last_draws);
+        s.theta_buf = (double*)(b + y.theta_buf);
+        s.Nmax = c->Nmax;
+        s.tiles_max = y.tiles_max;
+        s.Mmax = c->Mmax;
+        c->theta_cnt = (unsigned*)(b + y.theta_cnt);
+        c->score_out = (double*)(b + y.score_out);
+        if ((st = enter(c))) break;
+        if (cudaMemsetAsync(c->ws, 0, y.total, c->work) != cudaSuccess) { st = fail(c, MPCGS_E_CUDA, "memset"); break; }
+        std::vector<uint8_t> padded((size_t)n * c->Lpad, 0);
+        for (int i = 0; i < n; ++i) std::memcpy(padded.data() + (size_t)i * c->Lpad, codes.data() + (size_t)i * L, L);
+        if (cudaMemcpyAsync((void*)s.codes, padded.data(), padded.size(), cudaMemcpyHostToDevice, c->work) != cudaSuccess) {
+            st = fail(c, MPCGS_E_CUDA, "codes upload");
+            break;
+        }
+        if ((st = upload_state(c, parent.data(), age.data()))) break;
+        if (c->world > 1) {
+            NcclApi& api = nccl();
+            if (!api.ok || !cfg->nccl_id) { st = fail(c, MPCGS_E_NCCL, "NCCL unavailable or nccl_id missing"); break; }
+            ncclUniqueId id;
+            std::memcpy(&id, cfg->nccl_id, sizeof(id));
+            ncclResult_t r = api.commInitRank(&c->comm, c->world, id, c->rank);
+            if (r != ncclSuccess) { st = fail(c, MPCGS_E_NCCL, "ncclCommInitRank failed"); break; }
+        }
+        st = leave(c);
+    } while (0);
+    if (st != MPCGS_OK) {
+        // keep the context so that mpcgs_last_error can explain; caller frees it
+        *out = c;
+        return st;
+    }
+    *out = c;
+    return MPCGS_OK;
+}
+
+mpcgs_status mpcgs_init_phylip(const char* path, const mpcgs_config* cfg, double theta0, mpcgs_ctx** out) {
+    int32_t n, L;
+    if (mpcgs_phylip_dims(path, &n, &L) != MPCGS_OK) return MPCGS_E_ALIGNMENT;
+    std::vector<char> buf((size_t)n * L);
+    mpcgs_status st = mpcgs_phylip_read(path, buf.data(), (int32_t)buf.size());
+    if (st) return st;
+    std::vector<const char*> rows(n);
+    for (int i = 0; i < n; ++i) rows[i] = buf.data() + (size_t)i * L;
+    mpcgs_alignment a{n, L, rows.data()};
+    return mpcgs_init(&a, cfg, theta0, out);
+}
+
+mpcgs_status mpcgs_set_timing(mpcgs_ctx* c, int32_t on) {
+    CHECK_CTX(c);
+    c->timing = on != 0;
+    return MPCGS_OK;
+}
+
+mpcgs_status mpcgs_sample(mpcgs_ctx* c, int32_t N, int64_t M, uint64_t seed) {
+    CHECK_CTX(c);
+    if (N < 1 || N > c->Nmax || N % c->world != 0 || M < 0 || M > c->Mmax)
+        return fail(c, MPCGS_E_ARG, "n_proposals / n_samples out of range or not divisible by world");
+    const int64_t steps = (int64_t)c->burnin + (M + N - 1) / N;
+    mpcgs_status st = enter(c);
+    if (st) return st;
+    CU(cudaMemsetAsync(c->s.counters, 0, 8 * 8, c->work));
+    c->launches = 1;
+    const bool timed = c->timing;
+    if (timed) {
+        size_t need = (size_t)(2 * steps);
+        while (c->evpool.size() < need) {
+            cudaEvent_t ev;
+            CU(cudaEventCreate(&ev));
+            c->evpool.push_back(ev);
+        }
+    }
+    CU(cudaEventRecord(c->ev_b, c->work));
+    cudaEvent_t ev_end;
+    CU(cudaEventCreate(&ev_end));
+    for (int64_t s = 0; s < steps; ++s) {
+        if ((st = step_local_launch(c, seed, -1, N, timed, (int)s))) return st;
+        if ((st = allgather_records(c, N))) return st;
+        CU(launch_draw(c->s, seed, -1, N, -1, c->burnin, M, c->work));
+        ++c->launches;
+    }
+    CU(cudaEventRecord(ev_end, c->work));
+    CU(cudaEventSynchronize(ev_end));
+    float ms = 0.f;
+    CU(cudaEventElapsedTime(&ms, c->ev_b, ev_end));
+    cudaEventDestroy(ev_end);
+    c->loop_ms = ms;
+    c->prune_ms = 0.0;
+    if (timed)
+        for (int64_t s = 0; s < steps; ++s) {
+            float t = 0.f;
+            CU(cudaEventElapsedTime(&t, c->evpool[2 * s], c->evpool[2 * s + 1]));
+            c->prune_ms += t;
+        }
+    if ((st = check_status(c))) return st;
+    c->nsamples = M;
+    c->lastN = N;
+    c->sample_theta0 = c->s.theta0;
+    return MPCGS_OK;
+}
+
+mpcgs_status mpcgs_last_timing(const mpcgs_ctx* c, double* loop_ms, double* prune_ms, int64_t* launches) {
+    if (!c) return MPCGS_E_ARG;
+    if (loop_ms) *loop_ms = c->loop_ms;
+    if (prune_ms) *prune_ms = c->prune_ms;
+    if (launches) *launches = c->launches;
+    return MPCGS_OK;
+}
+
+int64_t mpcgs_num_samples(const mpcgs_ctx* c) { return c ? c->nsamples : 0; }
+
+mpcgs_status mpcgs_get_samples(mpcgs_ctx* c, int64_t first, int64_t count, double* S, double* logL, int64_t* step,
+                               int32_t* slot) {
+    CHECK_CTX(c);
+    if (first < 0 || count < 0 || first + count > c->nsamples) return fail(c, MPCGS_E_ARG, "sample range");
+    if (count == 0) return MPCGS_OK;
+    if (S) CU(cudaMemcpy(S, c->s.sS + first, 8 * (size_t)count, cudaMemcpyDeviceToHost));
+    if (logL) CU(cudaMemcpy(logL, c->s.sL + first, 8 * (size_t)count, cudaMemcpyDeviceToHost));
+    if (step) CU(cudaMemcpy(step, c->s.sStep + first, 8 * (size_t)count, cudaMemcpyDeviceToHost));
+    if (slot) CU(cudaMemcpy(slot, c->s.sSlot + first, 4 * (size_t)count, cudaMemcpyDeviceToHost));
+    return MPCGS_OK;
+}
+
+mpcgs_status mpcgs_score_trees(mpcgs_ctx* c, int32_t n_trees, const int32_t* parent, const double* age,
+                               double* logL_out) {
+    CHECK_CTX(c);
+    if (n_trees < 0 || (n_trees > 0 && (!parent || !age || !logL_out))) return fail(c, MPCGS_E_ARG, "score_trees args");
+    mpcgs_status st = enter(c);
+    if (st) return st;
+    for (int t0 = 0; t0 < n_trees; t0 += c->Nmax) {
+        const int cnt = std::min(c->Nmax, n_trees - t0);
+        st = score_batch(c, cnt, parent + (size_t)t0 * c->nn, age + (size_t)t0 * c->nn, logL_out + t0);
+        if (st) return st;
+    }
+    return MPCGS_OK;
+}
+
+mpcgs_status mpcgs_set_state(mpcgs_ctx* c, const int32_t* parent, const double* age) {
+    CHECK_CTX(c);
+    if (!parent || !age) return fail(c, MPCGS_E_ARG, "set_state args");
+    mpcgs_status st = enter(c);
+    if (st) return st;
+    return upload_state(c, parent, age);
+}
+
+mpcgs_status mpcgs_get_state(mpcgs_ctx* c, int32_t* parent, double* age, double* logL, double* S) {
+    CHECK_CTX(c);
+    mpcgs_status st = enter(c);
+    if (st) return st;
+    double gen[2];
+    if (parent) CU(cudaMemcpyAsync(parent, c->s.parent, 4 * (size_t)c->nn, cudaMemcpyDeviceToHost, c->work));
+    if (age) CU(cudaMemcpyAsync(age, c->s.age, 8 * (size_t)c->nn, cudaMemcpyDeviceToHost, c->work));
+    CU(cudaMemcpyAsync(gen, c->s.gen, 16, cudaMemcpyDeviceToHost, c->work));
+    if ((st = leave(c))) return st;
+    if (logL) *logL = gen[0];
+    if (S) *S = gen[1];
+    return MPCGS_OK;
+}
+
+mpcgs_status mpcgs_step_local(mpcgs_ctx* c, int64_t step, int32_t N, uint64_t seed) {
+    CHECK_CTX(c);
+    if (N < 1 || N > c->Nmax || N % c->world != 0 || step < 0) return fail(c, MPCGS_E_ARG, "step_local args");
+    mpcgs_status st = enter(c);
+    if (st) return st;
+    if ((st = step_local_launch(c, seed, step, N, false, 0))) return st;
+    if ((st = leave(c))) return st;
+    return check_status(c);
+}
+
+mpcgs_status mpcgs_get_records(mpcgs_ctx* c, int32_t first, int32_t count, double* host_rec) {
+    CHECK_CTX(c);
+    if (first < 0 || count < 0 || first + count > c->Nmax + 1 || (count && !host_rec)) return fail(c, MPCGS_E_ARG, "records range");
+    if (count) CU(cudaMemcpy(host_rec, c->s.rec + (size_t)first * REC, 8 * REC * (size_t)count, cudaMemcpyDeviceToHost));
+    return MPCGS_OK;
+}
+
+mpcgs_status mpcgs_put_records(mpcgs_ctx* c, int32_t first, int32_t count, const double* host_rec) {
+    CHECK_CTX(c);
+    if (first < 1 || count < 0 || first + count > c->Nmax + 1 || (count && !host_rec)) return fail(c, MPCGS_E_ARG, "records range");
+    if (count) CU(cudaMemcpy(c->s.rec + (size_t)first * REC, host_rec, 8 * REC * (size_t)count, cudaMemcpyHostToDevice));
+    return MPCGS_OK;
+}
+
+mpcgs_status mpcgs_step_finish(mpcgs_ctx* c, int64_t step, int32_t N, int32_t K, uint64_t seed, int32_t* draws) {
+    CHECK_CTX(c);
+    if (N < 1 || N > c->Nmax || K < 1 || K > N || step < 0) return fail(c, MPCGS_E_ARG, "step_finish args");
+    mpcgs_status st = enter(c);
+    if (st) return st;
+    CU(cudaMemsetAsync(c->s.counters + 2, 0, 8, c->work));
+    CU(launch_draw(c->s, seed, step, N, K, 0, 0, c->work));
+    if (draws) CU(cudaMemcpyAsync(draws, c->s.last_draws, 4 * (size_t)K, cudaMemcpyDeviceToHost, c->work));
+    if ((st = leave(c))) return st;
+    return check_status(c);
+}
+
+mpcgs_status mpcgs_step_trace(mpcgs_ctx* c, int64_t step, int32_t N, int32_t K, uint64_t seed, int32_t* target,
+                              double* logL, double* S, double* t12, int32_t* pair, int32_t* draws) {
+    CHECK_CTX(c);
+    if (c->world != 1) return fail(c, MPCGS_E_STATE, "step_trace needs world = 1 (use step_local/finish)");
+    if (N < 1 || N > c->Nmax || K < 1 || K > N || step < 0) return fail(c, MPCGS_E_ARG, "step_trace args");
+    mpcgs_status st = enter(c);
+    if (st) return st;
+    CU(cudaMemsetAsync(c->s.counters + 2, 0, 8, c->work));
+    if ((st = step_local_launch(c, seed, step, N, false, 0))) return st;
+    CU(launch_draw(c->s, seed, step, N, K, 0, 0, c->work));
+    std::vector<double> rec((size_t)(N + 1) * REC);
+    int32_t ci[16];
+    CU(cudaMemcpyAsync(rec.data(), c->s.rec, rec.size() * 8, cudaMemcpyDeviceToHost, c->work));
+    CU(cudaMemcpyAsync(ci, c->s.ctx_i, sizeof(ci), cudaMemcpyDeviceToHost, c->work));
+    if (draws) CU(cudaMemcpyAsync(draws, c->s.last_draws, 4 * (size_t)K, cudaMemcpyDeviceToHost, c->work));
+    if ((st = leave(c))) return st;
+    if ((st = check_status(c))) return st;
+    if (target) *target = ci[0];
+    for (int i = 0; i <= N; ++i) {
+        const double* r = rec.data() + (size_t)i * REC;
+        if (logL) logL[i] = r[0];
+        if (S) S[i] = r[1];
+        if (t12) { t12[2 * i] = r[2]; t12[2 * i + 1] = r[3]; }
+        if (pair) pair[i] = (int32_t)r[4];
+    }
+    return MPCGS_OK;
+}
+
+mpcgs_status mpcgs_set_theta0(mpcgs_ctx* c, double theta0) {
+    CHECK_CTX(c);
+    if (!(theta0 > 0.0) || !std::isfinite(theta0)) return fail(c, MPCGS_E_ARG, "theta0 must be positive");
+    c->theta0 = theta0;
+    c->s.theta0 = theta0;
+    return MPCGS_OK;
+}
+
+mpcgs_status mpcgs_get_model(const mpcgs_ctx* c, double* pi, double* mu) {
+    if (!c) return MPCGS_E_ARG;
+    if (pi)
+        for (int i = 0; i < 4; ++i) pi[i] = c->s.pi[i];
+    if (mu) *mu = c->s.u;
+    return MPCGS_OK;
+}
+
+}  // extern "C"
+
+namespace {
+// weighted moments at theta about center (device), returns m0, m1, m2 and the shift used
+mpcgs_status moments(mpcgs_ctx* c, double theta, double center, double smin, double smax, double out[4]) {
+    const double th0 = c->sample_theta0;
+    const double b = 1.0 / theta - 1.0 / th0;
+    const double shift = b > 0.0 ? -smin * b : -smax * b;
+    double* buf = c->s.theta_buf;
+    double* part = buf + 2 * MPCGS_MAX_GRID;
+    double* o3 = part + 3 * 296;
+    CU(launch_theta_moments(c->s.sS, c->nsamples, th0, theta, shift, center, part, c->theta_cnt, o3, c->work));
+    double h[3];
+    CU(cudaMemcpyAsync(h, o3, 24, cudaMemcpyDeviceToHost, c->work));
+    CU(cudaStreamSynchronize(c->work));
+    out[0] = h[0];
+    out[1] = h[1];
+    out[2] = h[2];
+    out[3] = shift;
+    return MPCGS_OK;
+}
+
+mpcgs_status minmax(mpcgs_ctx* c, double& smin, double& smax) {
+    double* o2 = c->s.theta_buf + 2 * MPCGS_MAX_GRID + 3 * 296 + 4;
+    CU(launch_minmax(c->s.sS, c->nsamples, o2, c->work));
+    double h[2];
+    CU(cudaMemcpyAsync(h, o2, 16, cudaMemcpyDeviceToHost, c->work));
+    CU(cudaStreamSynchronize(c->work));
+    smin = h[0];
+    smax = h[1];
+    return MPCGS_OK;
+}
+}  // namespace
+
+extern "C" {
+
+mpcgs_status mpcgs_log_rel_likelihood(mpcgs_ctx* c, double theta, double* out) {
+    CHECK_CTX(c);
+    if (c->nsamples < 1) return fail(c, MPCGS_E_STATE, "no samples");
+    if (!(theta > 0.0) || !out) return fail(c, MPCGS_E_ARG, "theta must be positive");
+    mpcgs_status st = enter(c);
+    if (st) return st;
+    double smin, smax, m[4];
+    if ((st = minmax(c, smin, smax))) return st;
+    if ((st = moments(c, theta, 0.0, smin, smax, m))) return st;
+    *out = (double)(c->n - 1) * std::log(c->sample_theta0 / theta) + m[3] + std::log(m[0]) -
+           std::log((double)c->nsamples);
+    return MPCGS_OK;
+}
+
+mpcgs_status mpcgs_estimate_theta(mpcgs_ctx* c, double* theta_hat, int32_t G, double* grid_theta, double* grid_logL) {
+    CHECK_CTX(c);
+    if (c->nsamples < 1) return fail(c, MPCGS_E_STATE, "estimate_theta before sample");
+    if (!theta_hat || G < 3 || G > MPCGS_MAX_GRID) return fail(c, MPCGS_E_ARG, "n_grid must be in [3, 4096]");
+    mpcgs_status st = enter(c);
+    if (st) return st;
+    const int n = c->n;
+    double smin, smax;
+    if ((st = minmax(c, smin, smax))) return st;
+    if (smin == smax) {  // every stationary point is S/(n-1) (Appendix B)
+        *theta_hat = smin / (n - 1);
+        for (int g = 0; g < G; ++g) {
+            if (grid_theta) grid_theta[g] = *theta_hat;
+            if (grid_logL) grid_logL[g] = 0.0;
+        }
+        return MPCGS_OK;
+    }
+    const double lo = smin / (n - 1), hi = smax / (n - 1);
+    double* buf = c->s.theta_buf;
+    CU(launch_theta_grid(c->s.sS, c->nsamples, n, c->sample_theta0, lo, hi, G, smin, smax, buf, c->work));
+    std::vector<double> h(2 * (size_t)G);
+    CU(cudaMemcpyAsync(h.data(), buf, 16 * (size_t)G, cudaMemcpyDeviceToHost, c->work));
+    CU(cudaStreamSynchronize(c->work));
+    int best = 0;
+    for (int g = 1; g < G; ++g)
+        if (h[G + g] > h[G + best]) best = g;
+    if (grid_theta) std::copy(h.begin(), h.begin() + G, grid_theta);
+    if (grid_logL) std::copy(h.begin() + G, h.end(), grid_logL);
+    double blo = best > 0 ? h[best - 1] : lo, bhi = best < G - 1 ? h[best + 1] : hi;
+    if (best == 0) blo = lo;
+    if (best == G - 1) bhi = hi;
+    // f(theta) = S_w(theta) - (n-1) theta has the sign of d lnL / d theta
+    auto f_at = [&](double th, double& f, double& fp) -> mpcgs_status {
+        double m[4];
+        const double cen = (double)(n - 1) * th;
+        mpcgs_status s2 = moments(c, th, cen, smin, smax, m);
+        if (s2) return s2;
+        const double mean = m[1] / m[0];
+        f = mean;  // S_w - c with c = (n-1) theta
+        const double var = std::max(0.0, m[2] / m[0] - mean * mean);
+        fp = var / (th * th) - (double)(n - 1);
+        return MPCGS_OK;
+    };
+    double flo, fhi, dummy;
+    if ((st = f_at(blo, flo, dummy))) return st;
+    if ((st = f_at(bhi, fhi, dummy))) return st;
+    double th = h[best];
+    if (flo >= 0.0 && fhi <= 0.0) {
+        for (int it = 0; it < 200; ++it) {
+            double f, fp;
+            if ((st = f_at(th, f, fp))) return st;
+            if (f >= 0.0) blo = th;
+            else bhi = th;
+            double tn = (fp < 0.0) ? th - f / fp : 0.5 * (blo + bhi);
+            if (!(tn > blo && tn < bhi)) tn = 0.5 * (blo + bhi);
+            if (std::fabs(tn - th) <= 1e-14 * th || bhi - blo <= 1e-15 * bhi) {
+                th = tn;
+                break;
+            }
+            th = tn;
+        }
+    } else {
+        // golden-section search on ln L inside the bracket
+        auto ll = [&](double t, double& v) -> mpcgs_status {
+            double m[4];
+            mpcgs_status s2 = moments(c, t, 0.0, smin, smax, m);
+            if (s2) return s2;
+            v = (double)(n - 1) * std::log(c->sample_theta0 / t) + m[3] + std::log(m[0]);
+            return MPCGS_OK;
+        };
+        const double gr = 0.6180339887498949;
+        double a = blo, bb = bhi, x1 = bb - gr * (bb - a), x2 = a + gr * (bb - a), v1, v2;
+        if ((st = ll(x1, v1)) || (st = ll(x2, v2))) return st;
+        for (int it = 0; it < 200 && bb - a > 1e-15 * bb; ++it) {
+            if (v1 > v2) { bb = x2; x2 = x1; v2 = v1; x1 = bb - gr * (bb - a); if ((st = ll(x1, v1))) return st; }
+            else { a = x1; x1 = x2; v1 = v2; x2 = a + gr * (bb - a); if ((st = ll(x2, v2))) return st; }
+        }
+        th = 0.5 * (a + bb);
+    }
+    *theta_hat = th;
+    return MPCGS_OK;
+}
+
+const char* mpcgs_last_error(const mpcgs_ctx* c) { return c ? c->err.c_str() : "null context"; }
+
+void mpcgs_free(mpcgs_ctx* c) {
+    if (!c) return;
+    if (c->work) cudaStreamSynchronize(c->work);
+    if (c->comm && nccl().ok) nccl().commDestroy(c->comm);
+    for (cudaEvent_t e : c->evpool) cudaEventDestroy(e);
+    if (c->ev_a) cudaEventDestroy(c->ev_a);
+    if (c->ev_b) cudaEventDestroy(c->ev_b);
+    if (c->own_ws && c->ws) cudaFree(c->ws);
+    if (c->work) cudaStreamDestroy(c->work);
+    delete c;
+}
+
+}  // extern "C"

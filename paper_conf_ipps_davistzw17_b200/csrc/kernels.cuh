@@ -1,0 +1,44 @@
+// kernels.cuh -- launch interfaces of the device kernels (internal to the library).
+#pragma once
+#include <cuda_runtime.h>
+
+#include "common.cuh"
+
+namespace mpcgs {
+
+constexpr int PRUNE_THREADS = 128;
+
+struct PruneArgs {
+    const uint8_t* codes;
+    int Lpad, L, nops;
+    double pi[4];
+    const uint32_t* sched_op;  // [ntrees][nops]
+    const void* sched_e;       // [ntrees][nops] float4 / double4
+    int tiles, sites_per_cta;
+    double* tile_part;         // [ntrees][tiles]
+    uint32_t* tile_cnt;        // [ntrees], zero on entry, reset by the kernel
+    double* out;               // logL of tree t -> out[(out_first + t) * out_stride]
+    int out_first, out_stride;
+};
+
+int prune_depth_for(int n);
+cudaError_t launch_prune(const PruneArgs& a, int ntrees, int depth, int precision, cudaStream_t st);
+
+// step kernels (step.cu); step < 0 -> read the step index from counters[0]
+cudaError_t launch_context(const DevState& s, uint64_t seed, int64_t step, cudaStream_t st);
+cudaError_t launch_propose(const DevState& s, uint64_t seed, int64_t step, int slot_first, int count,
+                           cudaStream_t st);
+// draw: K < 0 -> loop mode (burn-in / sampling from counters, store, advance step)
+cudaError_t launch_draw(const DevState& s, uint64_t seed, int64_t step, int N, int K, int burnin,
+                        int64_t M, cudaStream_t st);
+cudaError_t launch_fill_gen_record(const DevState& s, cudaStream_t st);
+
+// theta kernels (theta.cu)
+cudaError_t launch_minmax(const double* S, int64_t M, double* out2, cudaStream_t st);
+cudaError_t launch_theta_grid(const double* S, int64_t M, int n, double theta0, double lo, double hi, int G,
+                              double smin, double smax, double* out, cudaStream_t st);
+cudaError_t launch_theta_moments(const double* S, int64_t M, double theta0, double theta, double shift,
+                                 double center, double* part, unsigned* cnt, double* out3,
+                                 cudaStream_t st);
+
+}  // namespace mpcgs

@@ -1,0 +1,705 @@
+// step.cu -- one generalized Metropolis-Hastings step on the device
+// (Alg. 1; Fig. 12), without host round trips:
+//
+//   k_context  (1 CTA)      target draw (4.3 L1079-1093, S7) and the shared
+//                           neighbourhood context: feasible intervals, inactive
+//                           lineage counts, closed-form transition weights and
+//                           the backward messages P_i(n) (4.2 L986-1027, S9-S12)
+//   k_propose  (1 warp/slot) forward walk + event placement (4.2 L1028-1043,
+//                           S13-S15), tree patch, S_G (Eq. 18), Sethi-Ullman
+//                           register schedule for the pruning kernel
+//   k_draw     (1 CTA)      weights = softmax(logL) over N+1 states (Eq. 29-31,
+//                           S18: the prior is recorded, never added), K inverse-
+//                           CDF draws (L1140-1144), sample store, generator commit
+#include <cfloat>
+
+#include "common.cuh"
+#include "kernels.cuh"
+
+namespace mpcgs {
+
+constexpr int CTX_THREADS = 256;
+constexpr int DRAW_THREADS = 1024;
+
+// ------------------------------------------------------------------ helpers
+__device__ __forceinline__ int64_t step_of(const DevState& s, int64_t step_arg) {
+    return step_arg >= 0 ? step_arg : s.counters[0];
+}
+
+// Scaled weight W^_p(k -> kk) of an interval (length len, l inactive lineages):
+// every weight of the interval carries the common factor e^{r_1 len} (S12).
+__device__ double what(int k, int kk, double len, int l, double theta, bool inf) {
+    if (inf) return kk == 1 ? 1.0 : 0.0;  // unbounded root interval, l = 0 (S9)
+    const double r1 = (2.0 * l) / theta;
+    const double r2 = (2.0 + 4.0 * l) / theta;
+    const double r3 = (6.0 + 6.0 * l) / theta;
+    const double c2 = 2.0 / theta, c3 = 6.0 / theta;
+    if (k == 1) return kk == 1 ? 1.0 : 0.0;
+    if (k == 2) {
+        if (kk == 2) return exp(-(r2 - r1) * len);
+        if (kk == 1) return c2 * (-expm1(-(r2 - r1) * len)) / (r2 - r1);
+        return 0.0;
+    }
+    if (kk == 3) return exp(-(r3 - r1) * len);
+    if (kk == 2) return c3 * exp(-(r2 - r1) * len) * (-expm1(-(r3 - r2) * len)) / (r3 - r2);
+    const double a = (-expm1(-(r3 - r1) * len)) / (r3 - r1);
+    const double b = exp(-(r2 - r1) * len) * (-expm1(-(r3 - r2) * len)) / (r3 - r2);
+    return c3 * c2 * (a - b) / (r2 - r1);
+}
+
+// count of x[0..len) <= v (x sorted ascending)
+__device__ __forceinline__ int upper_count(const double* x, int len, double v) {
+    int lo = 0, hi = len;
+    while (lo < hi) {
+        int mid = (lo + hi) >> 1;
+        if (x[mid] <= v) lo = mid + 1;
+        else hi = mid;
+    }
+    return lo;
+}
+__device__ __forceinline__ int lower_count(const double* x, int len, double v) {
+    int lo = 0, hi = len;
+    while (lo < hi) {
+        int mid = (lo + hi) >> 1;
+        if (x[mid] < v) lo = mid + 1;
+        else hi = mid;
+    }
+    return lo;
+}
+
+// exclusive block scan of one int per thread; returns the prefix, total in *tot
+template <int NT>
+__device__ int block_exclusive_scan(int v, int* s_warp, int* tot) {
+    const int lane = threadIdx.x & 31, wid = threadIdx.x >> 5;
+    int x = v;
+#pragma unroll
+    for (int o = 1; o < 32; o <<= 1) {
+        int y = __shfl_up_sync(0xffffffffu, x, o);
+        if (lane >= o) x += y;
+    }
+    if (lane == 31) s_warp[wid] = x;
+    __syncthreads();
+    if (wid == 0) {
+        int w = lane < NT / 32 ? s_warp[lane] : 0;
+#pragma unroll
+        for (int o = 1; o < 32; o <<= 1) {
+            int y = __shfl_up_sync(0xffffffffu, w, o);
+            if (lane >= o) w += y;
+        }
+        if (lane < NT / 32) s_warp[lane] = w;
+    }
+    __syncthreads();
+    int base = wid > 0 ? s_warp[wid - 1] : 0;
+    *tot = s_warp[NT / 32 - 1];
+    __syncthreads();
+    return base + x - v;
+}
+
+// ------------------------------------------------------------------ k_context
+__global__ void __launch_bounds__(CTX_THREADS) k_context(DevState s, uint64_t seed, int64_t step_arg) {
+    extern __shared__ __align__(16) double csm[];
+    const int n = s.n, nn = s.nn, nint = n - 1;
+    double* sAge = csm;               // [n-1] ages of interior nodes (index v - n)
+    double* sF = sAge + nint;         // [n] sorted fixed ages
+    double* sX = sF + n;              // [n+1] merged cut candidates
+    double* sTau = sX + n + 1;        // [n+2]
+    double* sW = sTau + n + 2;        // [n][6] W^ rows: (1,1) (2,2) (2,1) (3,3) (3,2) (3,1)
+    double* sBeta = sW + 6 * n;       // [(n+1)][3]
+    int* sEntry = reinterpret_cast<int*>(sBeta + 3 * (n + 1));  // [n+1]
+    __shared__ int sh[16];
+    __shared__ double shd[8];
+    __shared__ int s_warp[CTX_THREADS / 32];
+    const int tid = threadIdx.x;
+
+    for (int i = tid; i < nint; i += CTX_THREADS) {
+        sAge[i] = s.age[n + i];
+        if (s.parent[n + i] < 0) sh[10] = n + i;  // root
+    }
+    __syncthreads();
+    if (tid == 0) {
+        const int64_t step = step_of(s, step_arg);
+        const int root = sh[10];
+        // target: uniform over the n-2 non-root interior nodes in id order (S7)
+        U4 w = philox(U4{0u, 0u, (uint32_t)step, TAG_TARGET}, (uint32_t)seed, (uint32_t)(seed >> 32));
+        int T = n + (int)__umulhi(w.x, (uint32_t)(n - 2));
+        if (T >= root) ++T;
+        const int Par = s.parent[T];
+        const int A = s.parent[Par];
+        const int sib = s.left[Par] == T ? s.right[Par] : s.left[Par];
+        int c[3] = {s.left[T], s.right[T], sib};
+        double a[3] = {s.age[c[0]], s.age[c[1]], s.age[c[2]]};
+        // sort the three children by (age, id)
+        for (int i = 0; i < 3; ++i)
+            for (int j = i + 1; j < 3; ++j)
+                if (a[j] < a[i] || (a[j] == a[i] && c[j] < c[i])) {
+                    int tc = c[i]; c[i] = c[j]; c[j] = tc;
+                    double ta = a[i]; a[i] = a[j]; a[j] = ta;
+                }
+        sh[0] = T; sh[1] = Par; sh[2] = A; sh[3] = A < 0; sh[4] = (a[2] == a[1]) ? 3 : 2;
+        sh[6] = c[0]; sh[7] = c[1]; sh[8] = c[2];
+        shd[0] = a[0]; shd[1] = a[1]; shd[2] = a[2];
+        shd[3] = A < 0 ? CUDART_INF : s.age[A];
+    }
+    __syncthreads();
+    const int T = sh[0], Par = sh[1];
+    const double a1 = shd[1], a2 = shd[2], tA = shd[3];
+    const bool rootcase = sh[3] != 0;
+    const int nfixed = n - 3;
+
+    // rank sort of the fixed interior nodes by (age, id)
+    for (int v = n + tid; v < nn; v += CTX_THREADS) {
+        if (v == T || v == Par) continue;
+        const double av = sAge[v - n];
+        int r = 0;
+        for (int w = n; w < nn; ++w) {
+            if (w == T || w == Par) continue;
+            const double aw = sAge[w - n];
+            r += (aw < av) || (aw == av && w < v);
+        }
+        sF[r] = av;
+    }
+    __syncthreads();
+    if (tid == 0) {
+        const int lo = upper_count(sF, nfixed, a1);  // fixed ages <= a(2): not cuts
+        const int hi = lower_count(sF, nfixed, tA);  // fixed ages <  t_A
+        const int has3 = a2 > a1;
+        sh[11] = lo;
+        sh[12] = hi - lo + has3;                    // merged candidate count
+        sh[13] = has3 ? lo + lower_count(sF + lo, hi - lo, a2) - lo : 0;  // insert position
+        sh[14] = has3;
+    }
+    __syncthreads();
+    const int lo = sh[11], cnt = sh[12], ins = sh[13], has3 = sh[14];
+    for (int j = tid; j < cnt; j += CTX_THREADS) {
+        double x;
+        if (!has3) x = sF[lo + j];
+        else if (j < ins) x = sF[lo + j];
+        else if (j == ins) x = a2;
+        else x = sF[lo + j - 1];
+        sX[j] = x;
+    }
+    __syncthreads();
+    // dedupe (equal ages are one cut) by an exclusive scan of keep flags
+    int carry = 0;
+    for (int base = 0; base < cnt; base += CTX_THREADS) {
+        const int j = base + tid;
+        const int keep = (j < cnt) && (j == 0 || sX[j] != sX[j - 1]);
+        int tot;
+        const int pos = block_exclusive_scan<CTX_THREADS>(keep, s_warp, &tot);
+        if (keep) sTau[1 + carry + pos] = sX[j];
+        carry += tot;
+    }
+    const int m = carry + 1;
+    if (tid == 0) {
+        sTau[0] = a1;
+        sTau[m] = tA;
+    }
+    __syncthreads();
+    // per-interval bookkeeping and closed-form weights
+    for (int p = tid; p < m; p += CTX_THREADS) {
+        const double tp = sTau[p];
+        const bool inf = rootcase && p == m - 1;
+        const double len = inf ? CUDART_INF : sTau[p + 1] - tp;
+        const int fixed_below = upper_count(sF, nfixed, tp);
+        const int kids_below = (shd[0] <= tp) + (a1 <= tp) + (a2 <= tp);
+        const int l = n - fixed_below - kids_below;
+        s.tau[p] = tp;
+        s.len[p] = len;
+        s.lcnt[p] = l;
+        sEntry[p] = (p >= 1 && has3 && tp == a2) ? 1 : 0;
+        const double th = s.theta0;
+        sW[p * 6 + 0] = what(1, 1, len, l, th, inf);
+        sW[p * 6 + 1] = what(2, 2, len, l, th, inf);
+        sW[p * 6 + 2] = what(2, 1, len, l, th, inf);
+        sW[p * 6 + 3] = what(3, 3, len, l, th, inf);
+        sW[p * 6 + 4] = what(3, 2, len, l, th, inf);
+        sW[p * 6 + 5] = what(3, 1, len, l, th, inf);
+    }
+    if (tid == 0) sEntry[m] = 0;
+    __syncthreads();
+    // backward messages (L1005-1020): exactly one lineage at the ancestor
+    if (tid == 0) {
+        double b1 = 1.0, b2 = 0.0, b3 = 0.0;
+        sBeta[m * 3 + 0] = b1; sBeta[m * 3 + 1] = b2; sBeta[m * 3 + 2] = b3;
+        for (int p = m - 1; p >= 0; --p) {
+            const int en = sEntry[p + 1];
+            // beta^end_p(k') = beta_{p+1}(k' + entry_{p+1})
+            const double e1 = en ? b2 : b1, e2 = en ? b3 : b2, e3 = en ? 0.0 : b3;
+            const double* W = sW + p * 6;
+            double n1 = W[0] * e1;
+            double n2 = W[1] * e2 + W[2] * e1;
+            double n3 = W[3] * e3 + W[4] * e2 + W[5] * e1;
+            const double mx = fmax(n1, fmax(n2, n3));
+            if (mx > 0.0 && (mx < 0x1p-500 || mx > 0x1p500)) {
+                const double f = exp2(-(double)ilogb(mx));   // exact power-of-two rescale
+                n1 *= f; n2 *= f; n3 *= f;
+            }
+            b1 = n1; b2 = n2; b3 = n3;
+            sBeta[p * 3 + 0] = b1; sBeta[p * 3 + 1] = b2; sBeta[p * 3 + 2] = b3;
+        }
+    }
+    __syncthreads();
+    // forward choice weights omega_p(k -> k') = W^_p(k -> k') beta_{p+1}(k' + entry_{p+1})
+    for (int p = tid; p < m; p += CTX_THREADS) {
+        const int en = sEntry[p + 1];
+        const double* bn = sBeta + (p + 1) * 3;
+        const double be1 = en ? bn[1] : bn[0], be2 = en ? bn[2] : bn[1], be3 = en ? 0.0 : bn[2];
+        const double* W = sW + p * 6;
+        double* om = s.omega + p * 9;
+        om[0] = W[0] * be1; om[1] = 0.0;         om[2] = 0.0;
+        om[3] = W[2] * be1; om[4] = W[1] * be2;  om[5] = 0.0;
+        om[6] = W[5] * be1; om[7] = W[4] * be2;  om[8] = W[3] * be3;
+        s.entry[p] = sEntry[p];
+    }
+    for (int i = tid; i < nfixed; i += CTX_THREADS) s.fixed[i] = sF[i];
+    if (tid == 0) {
+        s.tau[m] = tA;
+        s.entry[m] = 0;
+        for (int i = 0; i < 9; ++i) s.ctx_i[i] = sh[i];
+        s.ctx_i[5] = m;
+        s.ctx_i[9] = nfixed;
+        s.ctx_i[10] = sh[10];
+        for (int i = 0; i < 4; ++i) s.ctx_d[i] = shd[i];
+        s.counters[4] = T;
+    }
+}
+
+size_t context_smem_bytes(int n) {
+    return sizeof(double) * ((size_t)(n - 1) + n + (n + 1) + (n + 2) + 6 * n + 3 * (n + 1)) +
+           sizeof(int) * (n + 1) + 16;
+}
+
+cudaError_t launch_context(const DevState& s, uint64_t seed, int64_t step, cudaStream_t st) {
+    size_t smem = context_smem_bytes(s.n);
+    if (smem > 48 * 1024) {
+        cudaError_t e = cudaFuncSetAttribute(k_context, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+        if (e != cudaSuccess) return e;
+    }
+    k_context<<<1, CTX_THREADS, smem, st>>>(s, seed, step);
+    return cudaGetLastError();
+}
+
+// ------------------------------------------------------------------ k_propose
+// One event k -> k-1 in [0, len]: density prop. to e^{-delta s}; inverse CDF.
+__device__ double place_one(double len, double delta, double u, bool inf) {
+    if (inf) return -log(u) / delta;
+    double sv = -log1p(u * expm1(-delta * len)) / delta;
+    return fmin(fmax(sv, 0.0), len);
+}
+
+__device__ __forceinline__ double two_cdf(double x, double len, double A, double B) {
+    return (-expm1(-(A + B) * x)) / (A + B) - exp(-B * len) * (-expm1(-A * x)) / A;
+}
+
+// Two events 3 -> 1 in one interval: joint density e^{-A x - B y} on 0<x<y<len;
+// x by safeguarded Newton on its marginal CDF, then y | x by inversion (S13).
+__device__ void place_two(double len, double A, double B, double u1, double u2, bool inf, double& x,
+                          double& y) {
+    if (inf) {
+        x = -log(u1) / (A + B);
+        y = x - log(u2) / B;
+        return;
+    }
+    const double target = u1 * two_cdf(len, len, A, B);
+    double lo = 0.0, hi = len;
+    x = 0.5 * len;
+    for (int it = 0; it < 100; ++it) {
+        const double f = two_cdf(x, len, A, B) - target;
+        const double d = exp(-(A + B) * x) - exp(-B * len - A * x);
+        if (f > 0.0) hi = x;
+        else lo = x;
+        double xn = (d > 0.0) ? x - f / d : 0.5 * (lo + hi);
+        if (!(xn > lo && xn < hi)) xn = 0.5 * (lo + hi);
+        if (fabs(xn - x) <= 1e-15 * len) {
+            x = xn;
+            break;
+        }
+        x = xn;
+    }
+    y = x - log1p(u2 * expm1(-B * (len - x))) / B;
+    y = fmin(fmax(y, x), len);
+}
+
+struct Walk {
+    double t1, t2;
+    int pair, ok;
+};
+
+// Forward walk over the feasible intervals, young -> old (L1028-1034); RNG order
+// per interval: choice, event times, then the pair if the first coalescence
+// happens with three active lineages.
+__device__ Walk forward_walk(const DevState& s, int m, int k0, bool rootcase, uint64_t seed, uint32_t slot,
+                             uint32_t step) {
+    UStream us(seed, slot, step, TAG_PROPOSE);
+    Walk w{0.0, 0.0, 0, 0};
+    double tt[2] = {0.0, 0.0};
+    int k = k0, events = 0;
+    const double th = s.theta0;
+    for (int p = 0; p < m && events < 2; ++p) {
+        if (p >= 1) k += s.entry[p];
+        const bool inf = rootcase && p == m - 1;
+        const int l = s.lcnt[p];
+        const double r1 = (2.0 * l) / th, r2 = (2.0 + 4.0 * l) / th, r3 = (6.0 + 6.0 * l) / th;
+        const double* om = s.omega + p * 9 + (k - 1) * 3;
+        const double w0 = om[k - 1];
+        const double w1 = k >= 2 ? om[k - 2] : 0.0;
+        const double w2 = k >= 3 ? om[k - 3] : 0.0;
+        const double u = us.next();
+        const double total = (w0 + w1) + w2;
+        const double x = u * total;
+        int choice;
+        double cum = w0;
+        if (w0 > 0.0 && cum >= x) choice = 0;
+        else {
+            cum += w1;
+            if (w1 > 0.0 && cum >= x) choice = 1;
+            else {
+                cum += w2;
+                if (w2 > 0.0 && cum >= x) choice = 2;
+                else choice = w2 > 0.0 ? 2 : (w1 > 0.0 ? 1 : 0);
+            }
+        }
+        const double len = s.len[p], t0 = s.tau[p];
+        if (choice == 1) {
+            const double rk = k == 3 ? r3 : (k == 2 ? r2 : r1);
+            const double rk1 = k == 3 ? r2 : r1;
+            tt[events] = t0 + place_one(len, rk - rk1, us.next(), inf);
+        } else if (choice == 2) {
+            const double u1 = us.next(), u2 = us.next();
+            double xo, yo;
+            place_two(len, r3 - r2, r2 - r1, u1, u2, inf, xo, yo);
+            tt[0] = t0 + xo;
+            tt[1] = t0 + yo;
+        }
+        for (int e = 0; e < choice; ++e) {
+            if (events == 0) {
+                if (k == 3) {
+                    const int pc = (int)(3.0 * us.next());
+                    w.pair = pc > 2 ? 2 : pc;
+                } else {
+                    w.pair = 0;
+                }
+            }
+            ++events;
+        }
+        k -= choice;
+    }
+    w.ok = events == 2;
+    w.t1 = tt[0];
+    w.t2 = tt[1];
+    return w;
+}
+
+template <typename E4, typename ET>
+__global__ void __launch_bounds__(32) k_propose(DevState s, uint64_t seed, int64_t step_arg, int slot_first) {
+    extern __shared__ __align__(16) int psm[];
+    const int n = s.n, nn = s.nn, nint = n - 1;
+    int* sL = psm;             // [n-1] children of interior nodes (index v - n)
+    int* sR = sL + nint;       // [n-1]
+    int* sNeed = sR + nint;    // [nn]
+    int* sStack = sNeed + nn;  // [2n]
+    __shared__ double sh_d[8];  // t1, t2, e/em of changed branches
+    __shared__ int sh_i[8];
+    const int lane = threadIdx.x;
+    const int slot = slot_first + blockIdx.x;  // global slot 1..N
+    const int local = blockIdx.x;
+    const int64_t step = step_of(s, step_arg);
+
+    const int T = s.ctx_i[0], Par = s.ctx_i[1], A = s.ctx_i[2];
+    const bool rootcase = s.ctx_i[3] != 0;
+    const int k0 = s.ctx_i[4], m = s.ctx_i[5];
+    const int c0 = s.ctx_i[6], c1 = s.ctx_i[7], c2 = s.ctx_i[8];
+    const int nfixed = s.ctx_i[9], root = s.ctx_i[10];
+
+    if (lane == 0) {
+        Walk w = forward_walk(s, m, k0, rootcase, seed, (uint32_t)slot, (uint32_t)step);
+        int pair = w.pair;
+        double t1 = w.t1, t2 = w.t2;
+        if (!w.ok) {
+            // cannot happen for a valid context; keep the generator's tree and flag it
+            atomicOr(reinterpret_cast<unsigned long long*>(s.counters + 2), (unsigned long long)STATUS_WALK);
+            const int sib = s.left[Par] == T ? s.right[Par] : s.left[Par];
+            pair = sib == c2 ? 0 : (sib == c1 ? 1 : 2);
+            t1 = s.age[T];
+            t2 = s.age[Par];
+        }
+        sh_i[0] = pair;
+        sh_d[0] = t1;
+        sh_d[1] = t2;
+    }
+    for (int i = lane; i < nint; i += 32) {
+        sL[i] = s.left[n + i];
+        sR[i] = s.right[n + i];
+    }
+    for (int i = lane; i < nn; i += 32) sNeed[i] = i < n ? 0 : s.need[i];
+    __syncwarp();
+    const int pair = sh_i[0];
+    const double t1 = sh_d[0], t2 = sh_d[1];
+    // pair code 0 = (c1,c2), 1 = (c1,c3), 2 = (c2,c3) (S14)
+    const int x = pair == 2 ? c1 : c0;
+    const int y = pair == 0 ? c1 : c2;
+    const int z = pair == 0 ? c2 : (pair == 1 ? c1 : c0);
+    const double u = s.u;
+    if (lane == 0) {
+        // younger new node keeps the target's id, older keeps the parent's (S15)
+        sL[T - n] = min(x, y);
+        sR[T - n] = max(x, y);
+        sL[Par - n] = min(T, z);
+        sR[Par - n] = max(T, z);
+        sNeed[T] = su_need(sNeed[x], sNeed[y]);
+        sNeed[Par] = su_need(sNeed[T], sNeed[z]);
+        for (int v = A; v >= 0; v = s.parent[v]) sNeed[v] = su_need(sNeed[sL[v - n]], sNeed[sR[v - n]]);
+    } else if (lane == 1) {
+        sh_d[2] = exp(-u * (t1 - s.age[x]));
+        sh_d[3] = -expm1(-u * (t1 - s.age[x]));
+    } else if (lane == 2) {
+        sh_d[4] = exp(-u * (t1 - s.age[y]));
+        sh_d[5] = -expm1(-u * (t1 - s.age[y]));
+    } else if (lane == 3) {
+        sh_d[6] = exp(-u * (t2 - s.age[z]));
+        sh_d[7] = -expm1(-u * (t2 - s.age[z]));
+    }
+    __shared__ double sh_e2[4];
+    if (lane == 4) {
+        sh_e2[0] = exp(-u * (t2 - t1));
+        sh_e2[1] = -expm1(-u * (t2 - t1));
+    } else if (lane == 5) {
+        const double lp = rootcase ? 0.0 : s.age[A] - t2;
+        sh_e2[2] = exp(-u * lp);
+        sh_e2[3] = -expm1(-u * lp);
+    }
+    // S_G of the proposal: merge of the sorted fixed ages with {t1, t2} (Eq. 18 via
+    // S = 2 sum_i (n - i) h_i over sorted coalescence ages)
+    double base = 0.0, shift = 0.0;
+    int cnt1 = 0, cnt2 = 0;
+    for (int q = lane; q < nfixed; q += 32) {
+        const double f = s.fixed[q];
+        base += (double)(n - (q + 1)) * f;
+        shift += (t1 < f ? f : 0.0) + (t2 < f ? f : 0.0);
+        cnt1 += f <= t1;
+        cnt2 += f <= t2;
+    }
+#pragma unroll
+    for (int o = 16; o > 0; o >>= 1) {
+        base += __shfl_xor_sync(0xffffffffu, base, o);
+        shift += __shfl_xor_sync(0xffffffffu, shift, o);
+        cnt1 += __shfl_xor_sync(0xffffffffu, cnt1, o);
+        cnt2 += __shfl_xor_sync(0xffffffffu, cnt2, o);
+    }
+    __syncwarp();
+    if (lane == 0) {
+        const int r1 = 1 + cnt1, r2 = 2 + cnt2;
+        const double S = 2.0 * (base - shift) + 2.0 * (double)(n - r1) * t1 + 2.0 * (double)(n - r2) * t2;
+        double* rec = s.rec + (size_t)slot * REC;
+        rec[1] = S;
+        rec[2] = t1;
+        rec[3] = t2;
+        rec[4] = (double)pair;
+        // post-order register schedule of the proposal tree
+        const double* ge = s.e;
+        const double* gem = s.em;
+        auto e_of = [&](int c, double& e, double& em) {
+            if (c == x) { e = sh_d[2]; em = sh_d[3]; }
+            else if (c == y) { e = sh_d[4]; em = sh_d[5]; }
+            else if (c == z) { e = sh_d[6]; em = sh_d[7]; }
+            else if (c == T) { e = sh_e2[0]; em = sh_e2[1]; }
+            else if (c == Par) { e = sh_e2[2]; em = sh_e2[3]; }
+            else { e = ge[c]; em = gem[c]; }
+        };
+        uint32_t* op_out = s.sched_op + (size_t)local * s.nops;
+        E4* e_out = reinterpret_cast<E4*>(s.sched_e) + (size_t)local * s.nops;
+        emit_schedule(
+            n, root, [&](int v) { return sL[v - n]; }, [&](int v) { return sR[v - n]; },
+            [&](int v) { return sNeed[v]; },
+            [&](int i, uint32_t code, int ca, int cb) {
+                double ea, ema, eb, emb;
+                e_of(ca, ea, ema);
+                e_of(cb, eb, emb);
+                op_out[i] = code;
+                E4 v;
+                v.x = (ET)ea; v.y = (ET)ema; v.z = (ET)eb; v.w = (ET)emb;
+                e_out[i] = v;
+            },
+            sStack);
+    }
+}
+
+size_t propose_smem_bytes(int n) { return sizeof(int) * ((size_t)2 * (n - 1) + (2 * n - 1) + 2 * n); }
+
+cudaError_t launch_propose(const DevState& s, uint64_t seed, int64_t step, int slot_first, int count,
+                           cudaStream_t st) {
+    if (count <= 0) return cudaSuccess;
+    size_t smem = propose_smem_bytes(s.n);
+    if (s.precision == 32)
+        k_propose<float4, float><<<count, 32, smem, st>>>(s, seed, step, slot_first);
+    else
+        k_propose<double4, double><<<count, 32, smem, st>>>(s, seed, step, slot_first);
+    return cudaGetLastError();
+}
+
+// ------------------------------------------------------------------ k_draw
+__global__ void __launch_bounds__(DRAW_THREADS) k_draw(DevState s, uint64_t seed, int64_t step_arg, int N,
+                                                       int K_arg, int burnin, int64_t M) {
+    extern __shared__ __align__(16) double dsm[];
+    double* sC = dsm;  // [N+1] cumulative weights
+    __shared__ double s_red[DRAW_THREADS / 32];
+    __shared__ double s_max;
+    __shared__ int s_K, s_store;
+    const int tid = threadIdx.x, lane = tid & 31, wid = tid >> 5;
+    const int64_t step = step_of(s, step_arg);
+    const int nslots = N + 1;
+    const int T = s.ctx_i[0], Par = s.ctx_i[1];
+    if (tid == 0) {
+        // slot 0 = the generator with its cached likelihood (S16)
+        double* r0 = s.rec;
+        r0[0] = s.gen[0];
+        r0[1] = s.gen[1];
+        r0[2] = s.age[T];
+        r0[3] = s.age[Par];
+        r0[4] = -1.0;
+    }
+    __syncthreads();
+    const int chunk = (nslots + DRAW_THREADS - 1) / DRAW_THREADS;
+    const int i0 = tid * chunk, i1 = min(nslots, i0 + chunk);
+    double mx = -CUDART_INF;
+    for (int i = i0; i < i1; ++i) mx = fmax(mx, s.rec[(size_t)i * REC]);
+#pragma unroll
+    for (int o = 16; o > 0; o >>= 1) mx = fmax(mx, __shfl_xor_sync(0xffffffffu, mx, o));
+    if (lane == 0) s_red[wid] = mx;
+    __syncthreads();
+    if (tid == 0) {
+        double m2 = -CUDART_INF;
+        for (int w = 0; w < DRAW_THREADS / 32; ++w) m2 = fmax(m2, s_red[w]);
+        s_max = m2;
+        int K;
+        int store;
+        if (K_arg >= 0) {
+            K = K_arg;
+            store = 0;
+        } else if (step < burnin) {
+            K = 1;  // burn-in: one draw per set, not stored (Fig. 12)
+            store = 0;
+        } else {
+            const int64_t rem = M - s.counters[1];
+            K = (int)(rem < N ? rem : N);  // Alg. 1: N draws per set (S17)
+            store = 1;
+        }
+        s_K = K;
+        s_store = store;
+    }
+    __syncthreads();
+    mx = s_max;
+    if (!(mx > -CUDART_INF) || !(mx < CUDART_INF)) {  // all weights zero or NaN (S6)
+        if (tid == 0) {
+            atomicOr(reinterpret_cast<unsigned long long*>(s.counters + 2), (unsigned long long)STATUS_NUMERIC);
+            if (K_arg < 0) s.counters[0] = step + 1;
+        }
+        return;
+    }
+    // w_i = exp(logL_i - max): Eq. 31, proportional to P(D|G_i); inclusive scan in slot order
+    double run = 0.0;
+    for (int i = i0; i < i1; ++i) {
+        run += exp(s.rec[(size_t)i * REC] - mx);
+        sC[i] = run;
+    }
+    double x = run;
+#pragma unroll
+    for (int o = 1; o < 32; o <<= 1) {
+        double y = __shfl_up_sync(0xffffffffu, x, o);
+        if (lane >= o) x += y;
+    }
+    __syncthreads();
+    if (lane == 31) s_red[wid] = x;
+    __syncthreads();
+    if (wid == 0) {
+        double v = s_red[lane];
+#pragma unroll
+        for (int o = 1; o < 32; o <<= 1) {
+            double y = __shfl_up_sync(0xffffffffu, v, o);
+            if (lane >= o) v += y;
+        }
+        s_red[lane] = v;
+    }
+    __syncthreads();
+    const double before = (wid > 0 ? s_red[wid - 1] : 0.0) + (x - run);
+    for (int i = i0; i < i1; ++i) sC[i] += before;
+    __syncthreads();
+    const int K = s_K;
+    const double total = sC[N];
+    const int64_t stored = s.counters[1];
+    for (int d = tid; d < K; d += DRAW_THREADS) {
+        const double u = uniform_at(seed, 0u, (uint32_t)step, TAG_DRAW, (uint32_t)d);
+        const double xd = u * total;
+        int lo = 0, hi = N;  // lowest i with C_i >= x (L1140-1144)
+        while (lo < hi) {
+            const int mid = (lo + hi) >> 1;
+            if (sC[mid] >= xd) hi = mid;
+            else lo = mid + 1;
+        }
+        s.last_draws[d] = lo;
+        if (s_store) {
+            const int64_t j = stored + d;
+            const double* r = s.rec + (size_t)lo * REC;
+            s.sS[j] = r[1];
+            s.sL[j] = r[0];
+            s.sStep[j] = step;
+            s.sSlot[j] = lo;
+        }
+    }
+    __syncthreads();
+    if (tid != 0) return;
+    // commit: the last draw generates the next proposal set (Fig. 12)
+    const int I = K > 0 ? s.last_draws[K - 1] : 0;
+    if (I > 0) {
+        const double* r = s.rec + (size_t)I * REC;
+        const int A = s.ctx_i[2];
+        const int c0 = s.ctx_i[6], c1 = s.ctx_i[7], c2 = s.ctx_i[8];
+        const int pair = (int)r[4];
+        const double t1 = r[2], t2 = r[3], u = s.u;
+        const int x = pair == 2 ? c1 : c0;
+        const int y = pair == 0 ? c1 : c2;
+        const int z = pair == 0 ? c2 : (pair == 1 ? c1 : c0);
+        const int n = s.n;
+        s.left[T] = min(x, y);
+        s.right[T] = max(x, y);
+        s.left[Par] = min(T, z);
+        s.right[Par] = max(T, z);
+        s.parent[x] = T;
+        s.parent[y] = T;
+        s.parent[z] = Par;
+        s.parent[T] = Par;
+        s.age[T] = t1;
+        s.age[Par] = t2;
+        s.e[x] = exp(-u * (t1 - s.age[x]));
+        s.em[x] = -expm1(-u * (t1 - s.age[x]));
+        s.e[y] = exp(-u * (t1 - s.age[y]));
+        s.em[y] = -expm1(-u * (t1 - s.age[y]));
+        s.e[z] = exp(-u * (t2 - s.age[z]));
+        s.em[z] = -expm1(-u * (t2 - s.age[z]));
+        s.e[T] = exp(-u * (t2 - t1));
+        s.em[T] = -expm1(-u * (t2 - t1));
+        const double lp = A < 0 ? 0.0 : s.age[A] - t2;
+        s.e[Par] = exp(-u * lp);
+        s.em[Par] = -expm1(-u * lp);
+        auto nd = [&](int v) { return v < n ? 0 : s.need[v]; };
+        s.need[T] = su_need(nd(x), nd(y));
+        s.need[Par] = su_need(nd(T), nd(z));
+        for (int v = A; v >= 0; v = s.parent[v]) s.need[v] = su_need(nd(s.left[v]), nd(s.right[v]));
+        s.gen[0] = r[0];
+        s.gen[1] = r[1];
+    }
+    if (K_arg < 0) {
+        s.counters[0] = step + 1;
+        if (s_store) s.counters[1] = stored + K;
+    }
+    s.counters[3] = K;
+}
+
+cudaError_t launch_draw(const DevState& s, uint64_t seed, int64_t step, int N, int K, int burnin, int64_t M,
+                        cudaStream_t st) {
+    size_t smem = sizeof(double) * (size_t)(N + 1);
+    k_draw<<<1, DRAW_THREADS, smem, st>>>(s, seed, step, N, K, burnin, M);
+    return cudaGetLastError();
+}
+
+}  // namespace mpcgs

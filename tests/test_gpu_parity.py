@@ -1,0 +1,222 @@
+"""GPU parity of the CUDA path against the oracle, through the C ABI
+(BASELINE.json north_star tolerances):
+
+* per-genealogy ln P(D|G): 1e-9 relative (FP64 partials), 1e-4 (FP32);
+* target, interval choices/pair codes and draw indices bit-exact (draws flagged
+  near a threshold by the oracle are skipped), event times 1e-12 relative to
+  the tree height, S_G 1e-12;
+* theta-hat 1e-6 relative.
+"""
+import numpy as np
+import pytest
+
+import synth
+
+pytestmark = pytest.mark.gpu
+
+LL_TOL = {64: 1e-9, 32: 1e-4}
+
+
+@pytest.fixture(scope="module")
+def P():
+    import torch
+
+    if not torch.cuda.is_available():
+        pytest.skip("no CUDA device")
+    import paper_conf_ipps_davistzw17_b200 as pkg
+
+    pkg.lib()
+    return pkg
+
+
+def _ctx(P, codes, theta0, tree=None, **kw):
+    return P.Context(synth.to_strings(codes), theta0, init_tree=tree, **kw)
+
+
+# ------------------------------------------------------------------ pruning
+@pytest.mark.parametrize("precision", [64, 32])
+@pytest.mark.parametrize("n,L", [(3, 1), (4, 100), (12, 1000), (24, 129), (64, 1000), (128, 257), (256, 2000)])
+def test_score_trees_matches_oracle(P, orc, precision, n, L):
+    rng = np.random.default_rng(7 * n + L)
+    pi = np.array([0.22, 0.28, 0.31, 0.19])
+    u = orc.default_rate(pi)
+    true_p, true_a = synth.coalescent_tree(n, 0.05, rng)
+    codes = synth.f81_alignment(true_p, true_a, L, pi, u, rng)
+    trees = [synth.coalescent_tree(n, th, rng) for th in (0.01, 0.05, 0.3)]
+    trees += [synth.shaped_tree(n, s, rng, scale=0.02) for s in ("caterpillar", "balanced")]
+    ctx = _ctx(P, codes, 0.05, tree=trees[0], precision=precision, base_freq=pi, mu=u, max_proposals=8,
+               max_samples=16)
+    got = ctx.mpcgs_score_trees(np.stack([t[0] for t in trees]), np.stack([t[1] for t in trees]))
+    for (p, a), g in zip(trees, got):
+        want = orc.log_likelihood(codes, p, a, pi, u)
+        assert abs(g - want) <= LL_TOL[precision] * abs(want), (g, want)
+
+
+def test_score_adversarial_branch_lengths(P, orc):
+    rng = np.random.default_rng(3)
+    n, L = 16, 300
+    pi = np.array([0.1, 0.4, 0.4, 0.1])
+    u = orc.default_rate(pi)
+    codes = synth.random_alignment(n, L, rng, pi)
+    trees = []
+    for scale in (1e-9, 1e3, 0.0):
+        p, a = synth.shaped_tree(n, "random", rng, scale=1.0)
+        a = a * scale if scale > 0 else np.zeros_like(a)
+        trees.append((p, a))
+    p, a = synth.shaped_tree(n, "caterpillar", rng)
+    a[n:] = np.arange(1, n) * 1e-9          # tiny steps
+    trees.append((p, a))
+    ctx = _ctx(P, codes, 0.05, tree=trees[1], base_freq=pi, mu=u, max_proposals=8, max_samples=16)
+    got = ctx.mpcgs_score_trees(np.stack([t[0] for t in trees]), np.stack([t[1] for t in trees]))
+    for (p, a), g in zip(trees, got):
+        want = orc.log_likelihood(codes, p, a, pi, u)
+        if np.isinf(want):
+            assert g == want
+        else:
+            assert abs(g - want) <= 1e-9 * abs(want)
+
+
+def test_underflow_rescaling_long_alignment_many_tips(P, orc):
+    """P8: n = 256 tips with long branches forces per-node rescaling in both
+    precisions; sampled sites are checked one by one via L = 64 prefixes."""
+    rng = np.random.default_rng(5)
+    n, L = 256, 64
+    pi = np.array([0.05, 0.45, 0.45, 0.05])
+    u = orc.default_rate(pi)
+    p, a = synth.coalescent_tree(n, 5.0, rng)
+    codes = synth.random_alignment(n, L, rng, pi)
+    want = orc.log_likelihood(codes, p, a, pi, u)
+    assert want < -700 * 1.0  # per-site likelihoods far below FP32 range
+    for prec in (64, 32):
+        ctx = _ctx(P, codes, 0.05, tree=(p, a), base_freq=pi, mu=u, precision=prec, max_proposals=2,
+                   max_samples=4)
+        g = ctx.mpcgs_score_trees(p[None], a[None])[0]
+        assert abs(g - want) <= LL_TOL[prec] * abs(want)
+
+
+# ------------------------------------------------------------------ GMH step (lock-step, P20)
+def _lockstep(P, orc, wl, N, steps, seed, K=None, precision=64):
+    codes = wl["codes"]
+    pi = orc.base_freqs(codes)
+    u = orc.default_rate(pi)
+    theta0 = wl["theta0"]
+    parent, age = orc.upgma(codes, theta0)
+    gl = orc.log_likelihood(codes, parent, age, pi, u)
+    ctx = _ctx(P, codes, theta0, tree=(parent, age), precision=precision, max_proposals=N, max_samples=16)
+    K = N if K is None else K
+    height = age.max()
+    skipped = 0
+    for s in range(steps):
+        ctx.mpcgs_set_state(parent, age)
+        gp, ga, g_ll, g_S = ctx.mpcgs_get_state()
+        assert abs(g_ll - gl) <= LL_TOL[precision] * abs(gl)
+        tr = ctx.mpcgs_step_trace(s, N, K, seed)
+        ref = orc.gmh_step(codes, pi, u, theta0, N, K, seed, s, parent, age, gl)
+        assert tr["target"] == ref["target"]
+        ok = ~ref["slot_flag"]
+        ok[0] = True
+        assert np.array_equal(tr["pair"][1:][ok[1:]], ref["pair"][1:][ok[1:]])
+        scale = max(height, ref["t12"].max())
+        assert np.allclose(tr["t12"][ok], ref["t12"][ok], rtol=0, atol=1e-12 * scale)
+        assert np.allclose(tr["S"][ok], ref["S"][ok], rtol=1e-12, atol=0)
+        assert np.all(np.abs(tr["logL"][ok] - ref["logL"][ok]) <= LL_TOL[precision] * np.abs(ref["logL"][ok]))
+        if precision == 64 and not ref["draw_flag"].any() and ok.all():
+            assert np.array_equal(tr["draws"], ref["draws"])
+        else:
+            skipped += 1
+        parent, age, gl = ref["parent"], ref["age"], ref["gen_logL"]
+        height = age.max()
+    return skipped
+
+
+def test_lockstep_c1(P, orc):
+    wl = synth.workload("c1")
+    assert _lockstep(P, orc, wl, 16, 40, wl["chain_seed"]) <= 2
+
+
+def test_lockstep_c2_shape(P, orc):
+    wl = synth.workload("c2", L=300)
+    assert _lockstep(P, orc, wl, 64, 12, wl["chain_seed"]) <= 1
+
+
+def test_lockstep_n24_ragged(P, orc):
+    wl = synth.workload("c3", L=257, N=48)
+    assert _lockstep(P, orc, wl, 48, 6, 77) <= 1
+
+
+def test_lockstep_fp32_loglik_only(P, orc):
+    wl = synth.workload("c1")
+    _lockstep(P, orc, wl, 16, 10, 5, precision=32)
+
+
+def test_root_case_and_n3(P, orc):
+    rng = np.random.default_rng(0)
+    wl = dict(codes=synth.random_alignment(3, 40, rng), theta0=0.2)
+    assert _lockstep(P, orc, wl, 8, 20, 9) <= 1
+
+
+# ------------------------------------------------------------------ free-running chain vs oracle
+def test_free_running_chain_c1(P, orc):
+    wl = synth.workload("c1")
+    codes = wl["codes"]
+    pi = orc.base_freqs(codes)
+    u = orc.default_rate(pi)
+    parent, age = orc.upgma(codes, wl["theta0"])
+    N, M, B = 16, 400, 8
+    ref = orc.run_chain(codes, pi, u, wl["theta0"], N, B, M, wl["chain_seed"], parent, age)
+    ctx = _ctx(P, codes, wl["theta0"], burnin_steps=B, max_proposals=N, max_samples=M)
+    ctx.mpcgs_sample(N, M, wl["chain_seed"])
+    got = ctx.mpcgs_get_samples()
+    assert ctx.mpcgs_num_samples() == M
+    # identical until the first near-threshold flag of the oracle (none expected here)
+    if ref["n_flagged"] == 0:
+        assert np.array_equal(got["slot"], ref["slot"])
+        assert np.array_equal(got["step"], ref["step"])
+        assert np.allclose(got["S"], ref["S"], rtol=1e-11)
+        assert np.all(np.abs(got["logL"] - ref["logL"]) <= 1e-9 * np.abs(ref["logL"]))
+
+
+# ------------------------------------------------------------------ theta MLE
+def test_theta_hat_matches_oracle(P, orc):
+    wl = synth.workload("c2", L=400)
+    codes = wl["codes"]
+    N, M = 64, 3000
+    ctx = _ctx(P, codes, wl["theta0"], burnin_steps=20, max_proposals=N, max_samples=M)
+    ctx.mpcgs_sample(N, M, 123)
+    S = ctx.mpcgs_get_samples()["S"]
+    th = ctx.mpcgs_estimate_theta(256)
+    want = orc.theta_hat(S, 12, wl["theta0"])
+    assert abs(th - want) <= 1e-6 * want
+    for t in (0.5 * th, th, 2 * th):
+        assert np.isclose(ctx.mpcgs_log_rel_likelihood(t), orc.log_rel_likelihood(S, 12, wl["theta0"], t),
+                          rtol=1e-10, atol=1e-10)
+
+
+def test_theta_hat_degenerate_single_value(P, orc):
+    wl = synth.workload("c1")
+    ctx = _ctx(P, wl["codes"], wl["theta0"], max_proposals=16, max_samples=16)
+    ctx.mpcgs_sample(16, 1, 3)
+    S = ctx.mpcgs_get_samples()["S"]
+    assert np.isclose(ctx.mpcgs_estimate_theta(64), S[0] / 3, rtol=1e-15)
+
+
+# ------------------------------------------------------------------ errors
+def test_argument_errors(P):
+    wl = synth.workload("c1")
+    rows = synth.to_strings(wl["codes"])
+    with pytest.raises(P.MpcgsError):
+        P.Context(rows[:2], 0.01)
+    with pytest.raises(P.MpcgsError):
+        P.Context(rows, -1.0)
+    bad = list(rows)
+    bad[1] = bad[1][:5] + "N" + bad[1][6:]
+    with pytest.raises(P.MpcgsError) as ei:
+        P.Context(bad, 0.01)
+    assert ei.value.status == -2
+    ctx = P.Context(rows, 0.01, max_proposals=16, max_samples=100)
+    with pytest.raises(P.MpcgsError):
+        ctx.mpcgs_estimate_theta()        # before sample -> E_STATE
+    with pytest.raises(P.MpcgsError):
+        ctx.mpcgs_sample(32, 10, 1)       # N above capacity
+    with pytest.raises(P.MpcgsError):
+        ctx.mpcgs_sample(16, 1000, 1)     # M above capacity
