@@ -1,0 +1,314 @@
+"""Benchmark of the mpcgs hot path: one GMH step = context + N proposals +
+pruning of all N proposals over all sites + weights/draws/commit.
+
+    python bench.py [--gpus N] [--steps K] [--warmup W] [--impl ours|reference]
+                    [--workload c5] [--L 100000] [--precision 64]
+
+Metric (BASELINE.json): site-node partial likelihoods scored per second (and
+proposal genealogies scored per second), whole job over all ranks.  Default
+workload: config c5 at its largest sweep point, 64 sequences x 100,000 bp,
+N = 1,024 proposals per step (the config on which the north star's scaling
+target is stated; it fits one GPU).  Inputs are synthetic: an ms-style
+coalescent tree at theta = 1 and F81 sequences with uniform pi (synth/).
+
+Timing: W untimed warm-up steps, then K steps timed on the device with CUDA
+events on the library's stream (step boundaries and every pruning launch),
+L2 flushed (256 MiB write) between timed steps outside the timed intervals;
+barrier + synchronize on both sides; max over ranks.  nvidia-smi samples the
+clocks during the timed region.  `--impl reference` times the plain CPU oracle
+(oracle/) on a bounded sample of the same workload.
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import subprocess
+import sys
+import tempfile
+import time
+
+import numpy as np
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+import synth  # noqa: E402
+
+METRIC = json.load(open(os.path.join(ROOT, "BASELINE.json")))["metric"]
+UNIT = "site-node partials/s"
+
+
+def flops_per_site(n: int) -> int:
+    """Algorithmic FP operations of one site of one genealogy:
+    tip child 2 (em*pi_x, +e), internal child 16 (pi.L 7, em*s 1, e*L+t 8),
+    node product 4; n tips, n-2 internal children, n-1 nodes."""
+    return 2 * n + 16 * (n - 2) + 4 * (n - 1)
+
+
+def peaks():
+    mp = {}
+    try:
+        mp = json.load(open(os.path.join(ROOT, "MEASURED_PEAKS.json")))
+    except Exception:
+        pass
+    mhz = float(mp.get("sm_max_mhz", 1965.0))
+    # B200: 148 SMs; per SM per clock 64 FP64 FMA lanes, 128 FP32 FMA lanes (FMA = 2 flops)
+    return {64: 148 * 64 * 2 * mhz * 1e6 / 1e12, 32: 148 * 128 * 2 * mhz * 1e6 / 1e12}, mhz, mp
+
+
+class Clocks:
+    def __init__(self, idx: int):
+        self.path = tempfile.mktemp(prefix="clk", suffix=".csv")
+        q = ("index,clocks.sm,clocks.max.sm,power.draw,clocks_event_reasons.active,"
+             "clocks_event_reasons.hw_slowdown,clocks_event_reasons.hw_thermal_slowdown,"
+             "clocks_event_reasons.sw_thermal_slowdown,clocks_event_reasons.sw_power_cap")
+        try:
+            self.p = subprocess.Popen(["nvidia-smi", f"--id={idx}", f"--query-gpu={q}", "--format=csv,noheader,nounits",
+                                       "-lms", "100"], stdout=open(self.path, "w"), stderr=subprocess.DEVNULL)
+        except Exception:
+            self.p = None
+
+    def stop(self):
+        if self.p is None:
+            return None
+        time.sleep(0.25)
+        self.p.terminate()
+        try:
+            self.p.wait(timeout=5)
+        except Exception:
+            self.p.kill()
+        rows = []
+        for ln in open(self.path):
+            f = [x.strip() for x in ln.split(",")]
+            if len(f) >= 9:
+                rows.append(f)
+        if not rows:
+            return None
+        sm = [float(r[1]) for r in rows if r[1].replace(".", "").isdigit()]
+        reasons = set()
+        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
+        for r in rows:
+            for k, nm in enumerate(names):
+                if r[5 + k].lower().startswith("active"):
+                    reasons.add(nm)
+        return {"sm_mhz": float(np.median(sm)) if sm else None, "sm_max_mhz": float(rows[0][2]),
+                "reasons": sorted(reasons), "samples": len(rows)}
+
+
+def traffic_from_profiles(tag: str):
+    p = os.path.join(ROOT, "profiles", "prune_traffic.json")
+    try:
+        d = json.load(open(p))
+        return d.get(tag)
+    except Exception:
+        return None
+
+
+def cpu_oracle_sample(wl, seconds: float, n_prop: int = 1):
+    """Time the oracle's GMH step on the same workload (bounded: n_prop proposals)."""
+    import oracle
+
+    codes = wl["codes"]
+    pi = oracle.base_freqs(codes)
+    u = oracle.default_rate(pi)
+    parent, age = wl["true_parent"], wl["true_age"]
+    gl = oracle.log_likelihood(codes, parent, age, pi, u)
+    n, L = codes.shape
+    steps, t0 = 0, time.perf_counter()
+    while True:
+        tr = oracle.gmh_step(codes, pi, u, wl["theta0"], n_prop, n_prop, wl["chain_seed"], steps, parent, age, gl)
+        parent, age, gl = tr["parent"], tr["age"], tr["gen_logL"]
+        steps += 1
+        if time.perf_counter() - t0 >= seconds:
+            break
+    dt = time.perf_counter() - t0
+    partials = steps * n_prop * L * (n - 1)
+    return partials / dt, steps, dt
+
+
+def run_reference(args, wl, rank):
+    if rank != 0:
+        return
+    codes = wl["codes"]
+    n, L = codes.shape
+    import oracle
+
+    pi = oracle.base_freqs(codes)
+    u = oracle.default_rate(pi)
+    parent, age = wl["true_parent"], wl["true_age"]
+    gl = oracle.log_likelihood(codes, parent, age, pi, u)
+    n_prop = 1
+    for s in range(args.warmup):
+        tr = oracle.gmh_step(codes, pi, u, wl["theta0"], n_prop, n_prop, wl["chain_seed"], s, parent, age, gl)
+        parent, age, gl = tr["parent"], tr["age"], tr["gen_logL"]
+    t0 = time.perf_counter()
+    for s in range(args.steps):
+        tr = oracle.gmh_step(codes, pi, u, wl["theta0"], n_prop, n_prop, wl["chain_seed"], args.warmup + s,
+                             parent, age, gl)
+        parent, age, gl = tr["parent"], tr["age"], tr["gen_logL"]
+    dt = time.perf_counter() - t0
+    partials = args.steps * n_prop * L * (n - 1)
+    value = partials / dt
+    sample = f"oracle GMH step with {n_prop} proposal (of {wl['N']}) over all {L} sites, {args.steps} steps"
+    line = {
+        "impl": "reference", "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": args.gpus,
+        "steps": args.steps, "warmup": args.warmup, "ms_per_step": 1e3 * dt / args.steps,
+        "higher_is_better": True, "scaling": "strong", "vs_baseline": None, "dtype": "f64", "data": "synthetic",
+        "config": workload_config(args, wl),
+        "cpu_baseline": {"value": value, "unit": UNIT, "cores": 1, "kind": "oracle", "sample": sample},
+        "e2e": {"value": value, "unit": UNIT, "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
+        "proposals_per_s": args.steps * n_prop / dt,
+    }
+    print(json.dumps(line), flush=True)
+
+
+def workload_config(args, wl):
+    n, L = wl["codes"].shape
+    return {"workload": f"{args.workload}: {n} sequences x {L} bp, {wl['N']} proposals/step, theta0 {wl['theta0']}",
+            "n_seq": n, "n_sites": L, "proposals_per_step": wl["N"], "theta0": wl["theta0"],
+            "precision": args.precision, "l2": "flushed (256 MiB write) between timed steps",
+            "parallelism": f"proposal-sharded x{args.gpus}", "init_tree": "synthetic true tree (ms-style)"}
+
+
+def main():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=20)
+    ap.add_argument("--warmup", type=int, default=5)
+    ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
+    ap.add_argument("--workload", default="c5")
+    ap.add_argument("--L", type=int, default=None)
+    ap.add_argument("--n", type=int, default=None)
+    ap.add_argument("--N", type=int, default=None)
+    ap.add_argument("--precision", type=int, default=64, choices=[32, 64])
+    ap.add_argument("--cpu-seconds", type=float, default=12.0)
+    ap.add_argument("--no-e2e", action="store_true")
+    args = ap.parse_args()
+    args.warmup = max(args.warmup, 3)
+
+    world = int(os.environ.get("WORLD_SIZE", "1"))
+    rank = int(os.environ.get("RANK", "0"))
+    local = int(os.environ.get("LOCAL_RANK", "0"))
+    over = {}
+    if args.L:
+        over["L"] = args.L
+    if args.n:
+        over["n"] = args.n
+    if args.N:
+        over["N"] = args.N
+    wl = synth.workload(args.workload, **over)
+    if args.impl == "reference":
+        run_reference(args, wl, rank)
+        return
+
+    import torch
+
+    import paper_conf_ipps_davistzw17_b200 as P
+
+    torch.cuda.set_device(local)
+    dist = None
+    nccl_id = None
+    if world > 1:
+        import torch.distributed as dist
+
+        dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+        idb = torch.zeros(128, dtype=torch.uint8, device="cuda")
+        if rank == 0:
+            idb.copy_(torch.frombuffer(bytearray(P.mpcgs_nccl_unique_id()), dtype=torch.uint8))
+        dist.broadcast(idb, 0)
+        nccl_id = bytes(idb.cpu().numpy().tobytes())
+
+    codes = wl["codes"]
+    n, L = codes.shape
+    N = wl["N"]
+    rows = synth.to_strings(codes)
+    total_steps = args.warmup + args.steps
+    stream = torch.cuda.current_stream().cuda_stream
+
+    def barrier():
+        if dist is not None:
+            dist.barrier()
+        torch.cuda.synchronize()
+
+    ctx = P.Context(rows, wl["theta0"], precision=args.precision, max_proposals=N, max_samples=N * total_steps,
+                    init_tree=(wl["true_parent"], wl["true_age"]), rank=rank, world=world, nccl_id=nccl_id,
+                    stream=stream)
+    # warm-up (untimed): W steps
+    ctx.mpcgs_sample(N, N * args.warmup, wl["chain_seed"])
+    ctx.mpcgs_set_timing(3)   # per-step + per-prune CUDA events, L2 flush between steps
+    barrier()
+    clk = Clocks(local)
+    ctx.mpcgs_sample(N, N * args.steps, wl["chain_seed"] + 1)
+    barrier()
+    clocks = clk.stop()
+    loop_ms, prune_ms, launches = ctx.mpcgs_last_timing()
+    t = torch.tensor([loop_ms, prune_ms], dtype=torch.float64, device="cuda")
+    if dist is not None:
+        dist.all_reduce(t, op=dist.ReduceOp.MAX)
+    loop_ms, prune_ms = float(t[0]), float(t[1])
+    partials = N * L * (n - 1) * args.steps
+    value = partials / (loop_ms / 1e3)
+    ms_per_step = loop_ms / args.steps
+
+    # roofline of the dominant kernel (prune): algorithmic flops per launch / mean launch time
+    pk, mhz, mp = peaks()
+    local_trees = N // world
+    flops_launch = local_trees * L * flops_per_site(n)
+    prune_avg_s = (prune_ms / 1e3) / args.steps
+    achieved = flops_launch / prune_avg_s / 1e12
+    roof = {"bound": "alu", "achieved": achieved, "peak": pk[args.precision], "unit": "TFLOP/s",
+            "frac": achieved / pk[args.precision], "traffic": traffic_from_profiles(f"{args.workload}_fp{args.precision}"),
+            "kernel": "k_prune", "prune_share_of_step": prune_ms / loop_ms,
+            "peak_source": f"derived: 148 SM x {'64 FP64' if args.precision == 64 else '128 FP32'} FMA lanes x 2 x "
+                           f"{mhz:.0f} MHz (MEASURED_PEAKS sm_max_mhz)",
+            "partials_per_s_prune_only": N * L * (n - 1) / (prune_avg_s * world) if world == 1 else
+            local_trees * L * (n - 1) / prune_avg_s}
+
+    # end-to-end through the public API from host buffers: init (H2D of the alignment
+    # and G0) + K steps + D2H of the samples, wall clock, max over ranks
+    e2e = None
+    if not args.no_e2e:
+        barrier()
+        t0 = time.perf_counter()
+        ctx2 = P.Context(rows, wl["theta0"], precision=args.precision, max_proposals=N, max_samples=N * args.steps,
+                         init_tree=(wl["true_parent"], wl["true_age"]), rank=rank, world=world, nccl_id=nccl_id,
+                         stream=stream)
+        ctx2.mpcgs_sample(N, N * args.steps, wl["chain_seed"] + 1)
+        smp = ctx2.mpcgs_get_samples()
+        barrier()
+        dt = time.perf_counter() - t0
+        ctx2.free()
+        tt = torch.tensor([dt], dtype=torch.float64, device="cuda")
+        if dist is not None:
+            dist.all_reduce(tt, op=dist.ReduceOp.MAX)
+        dt = float(tt[0])
+        h2d = n * L + (2 * n - 1) * 12
+        d2h = sum(v.nbytes for v in smp.values())
+        e2e = {"value": partials / dt, "unit": UNIT, "h2d_bytes_per_step": h2d / args.steps,
+               "d2h_bytes_per_step": d2h / args.steps, "includes": "init (alignment H2D, G0 scoring) + sampling + "
+               "sample D2H, wall clock"}
+
+    cpu = None
+    if rank == 0 and world == 1 and args.cpu_seconds > 0:
+        v, st, dt = cpu_oracle_sample(wl, args.cpu_seconds)
+        cpu = {"value": v, "unit": UNIT, "cores": 1, "kind": "oracle",
+               "sample": f"{st} oracle GMH steps with 1 proposal each over all {L} sites ({dt:.1f} s)"}
+
+    if rank == 0:
+        line = {
+            "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world, "steps": args.steps,
+            "warmup": args.warmup, "ms_per_step": ms_per_step, "higher_is_better": True, "scaling": "strong",
+            "vs_baseline": None, "dtype": "f64" if args.precision == 64 else "f32", "data": "synthetic",
+            "config": workload_config(args, wl), "proposals_per_s": N * args.steps / (loop_ms / 1e3),
+            "roofline": roof, "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": int(launches),
+            "clocks": clocks,
+        }
+        print(json.dumps(line), flush=True)
+    ctx.free()
+    if dist is not None:
+        dist.destroy_process_group()
+
+
+if __name__ == "__main__":
+    main()

@@ -73,8 +73,10 @@ struct mpcgs_ctx {
     bool sticky = false;
     std::string err;
     ncclComm_t comm = nullptr;
-    bool timing = false;
+    int timing = 0;              // bit 0: events per step / prune launch; bit 1: flush L2 between steps
+    void* flush_buf = nullptr;   // 256 MiB scratch written between timed steps (> 126 MB L2)
     double loop_ms = 0.0, prune_ms = 0.0;
+    int graph_steps = 32;
     int64_t launches = 0;
     std::vector<cudaEvent_t> evpool;
     cudaEvent_t ev_a = nullptr, ev_b = nullptr;
@@ -416,14 +418,15 @@ mpcgs_status check_status(mpcgs_ctx* c) {
 }
 
 // one step's proposal work for this rank: context, propose, prune
-mpcgs_status step_local_launch(mpcgs_ctx* c, uint64_t seed, int64_t step, int N, bool timed, int ev_idx) {
+mpcgs_status step_local_launch(mpcgs_ctx* c, uint64_t seed, int64_t step, int N, cudaEvent_t pre = nullptr,
+                               cudaEvent_t post = nullptr) {
     int first = 1 + c->rank * (N / c->world), count = N / c->world;
     CU(launch_context(c->s, seed, step, c->work));
     CU(launch_propose(c->s, seed, step, first, count, c->work));
     PruneArgs a = prune_args(c, count, c->s.rec, first, REC);
-    if (timed) CU(cudaEventRecord(c->evpool[2 * ev_idx], c->work));
+    if (pre) CU(cudaEventRecord(pre, c->work));
     CU(launch_prune(a, count, c->depth, c->precision, c->work));
-    if (timed) CU(cudaEventRecord(c->evpool[2 * ev_idx + 1], c->work));
+    if (post) CU(cudaEventRecord(post, c->work));
     c->launches += 3;
     return MPCGS_OK;
 }
@@ -731,9 +734,13 @@ mpcgs_status mpcgs_init_phylip(const char* path, const mpcgs_config* cfg, double
     return mpcgs_init(&a, cfg, theta0, out);
 }
 
-mpcgs_status mpcgs_set_timing(mpcgs_ctx* c, int32_t on) {
+mpcgs_status mpcgs_set_timing(mpcgs_ctx* c, int32_t mode) {
     CHECK_CTX(c);
-    c->timing = on != 0;
+    c->timing = mode & 3;
+    if ((c->timing & 2) && !c->flush_buf) {
+        if (cudaMalloc(&c->flush_buf, (size_t)256 << 20) != cudaSuccess)
+            return fail(c, MPCGS_E_NOMEM, "flush buffer allocation failed");
+    }
     return MPCGS_OK;
 }
 
@@ -745,38 +752,84 @@ mpcgs_status mpcgs_sample(mpcgs_ctx* c, int32_t N, int64_t M, uint64_t seed) {
     mpcgs_status st = enter(c);
     if (st) return st;
     CU(cudaMemsetAsync(c->s.counters, 0, 8 * 8, c->work));
-    c->launches = 1;
-    const bool timed = c->timing;
-    if (timed) {
-        size_t need = (size_t)(2 * steps);
+    c->launches = 0;
+    c->prune_ms = 0.0;
+    auto one_step = [&]() -> mpcgs_status {
+        mpcgs_status s2 = step_local_launch(c, seed, -1, N);
+        if (s2) return s2;
+        if ((s2 = allgather_records(c, N))) return s2;
+        CU(launch_draw(c->s, seed, -1, N, -1, c->burnin, M, c->work));
+        ++c->launches;
+        return MPCGS_OK;
+    };
+    if (c->timing & 1) {
+        // device-timed steps: events at step boundaries and around every pruning
+        // launch; optional L2 flush between steps, outside the timed intervals
+        const size_t need = (size_t)4 * steps;
         while (c->evpool.size() < need) {
             cudaEvent_t ev;
             CU(cudaEventCreate(&ev));
             c->evpool.push_back(ev);
         }
-    }
-    CU(cudaEventRecord(c->ev_b, c->work));
-    cudaEvent_t ev_end;
-    CU(cudaEventCreate(&ev_end));
-    for (int64_t s = 0; s < steps; ++s) {
-        if ((st = step_local_launch(c, seed, -1, N, timed, (int)s))) return st;
-        if ((st = allgather_records(c, N))) return st;
-        CU(launch_draw(c->s, seed, -1, N, -1, c->burnin, M, c->work));
-        ++c->launches;
-    }
-    CU(cudaEventRecord(ev_end, c->work));
-    CU(cudaEventSynchronize(ev_end));
-    float ms = 0.f;
-    CU(cudaEventElapsedTime(&ms, c->ev_b, ev_end));
-    cudaEventDestroy(ev_end);
-    c->loop_ms = ms;
-    c->prune_ms = 0.0;
-    if (timed)
-        for (int64_t s = 0; s < steps; ++s) {
-            float t = 0.f;
-            CU(cudaEventElapsedTime(&t, c->evpool[2 * s], c->evpool[2 * s + 1]));
-            c->prune_ms += t;
+        for (int64_t k = 0; k < steps; ++k) {
+            if ((c->timing & 2) && c->flush_buf)
+                CU(cudaMemsetAsync(c->flush_buf, (int)(k & 0xff), (size_t)256 << 20, c->work));
+            CU(cudaEventRecord(c->evpool[4 * k + 0], c->work));
+            if ((st = step_local_launch(c, seed, -1, N, c->evpool[4 * k + 1], c->evpool[4 * k + 2]))) return st;
+            if ((st = allgather_records(c, N))) return st;
+            CU(launch_draw(c->s, seed, -1, N, -1, c->burnin, M, c->work));
+            ++c->launches;
+            CU(cudaEventRecord(c->evpool[4 * k + 3], c->work));
         }
+        CU(cudaEventSynchronize(c->evpool[4 * (steps - 1) + 3]));
+        double tot = 0.0, pr = 0.0;
+        for (int64_t k = 0; k < steps; ++k) {
+            float t = 0.f, q = 0.f;
+            CU(cudaEventElapsedTime(&t, c->evpool[4 * k + 0], c->evpool[4 * k + 3]));
+            CU(cudaEventElapsedTime(&q, c->evpool[4 * k + 1], c->evpool[4 * k + 2]));
+            tot += t;
+            pr += q;
+        }
+        c->loop_ms = tot;
+        c->prune_ms = pr;
+    } else {
+        // CUDA graph of up to graph_steps steps, replayed; the kernels read the step
+        // counter from device memory, so one graph serves every step
+        const int64_t G = std::min<int64_t>(c->graph_steps, std::max<int64_t>(steps, 1));
+        cudaGraph_t graph = nullptr;
+        cudaGraphExec_t exec = nullptr;
+        const int64_t reps = steps / G, rest = steps % G;
+        if (reps > 0) {
+            CU(cudaStreamBeginCapture(c->work, cudaStreamCaptureModeThreadLocal));
+            for (int64_t k = 0; k < G; ++k) {
+                if ((st = one_step())) {
+                    cudaStreamEndCapture(c->work, &graph);
+                    if (graph) cudaGraphDestroy(graph);
+                    return st;
+                }
+            }
+            CU(cudaStreamEndCapture(c->work, &graph));
+            CU(cudaGraphInstantiate(&exec, graph, 0));
+            c->launches = 0;
+        }
+        CU(cudaEventRecord(c->ev_b, c->work));
+        for (int64_t r = 0; r < reps; ++r) {
+            CU(cudaGraphLaunch(exec, c->work));
+            c->launches += 4 * G;
+        }
+        for (int64_t k = 0; k < rest; ++k)
+            if ((st = one_step())) return st;
+        cudaEvent_t ev_end;
+        CU(cudaEventCreate(&ev_end));
+        CU(cudaEventRecord(ev_end, c->work));
+        CU(cudaEventSynchronize(ev_end));
+        float ms = 0.f;
+        CU(cudaEventElapsedTime(&ms, c->ev_b, ev_end));
+        cudaEventDestroy(ev_end);
+        if (exec) cudaGraphExecDestroy(exec);
+        if (graph) cudaGraphDestroy(graph);
+        c->loop_ms = ms;
+    }
     if ((st = check_status(c))) return st;
     c->nsamples = M;
     c->lastN = N;
@@ -847,7 +900,7 @@ mpcgs_status mpcgs_step_local(mpcgs_ctx* c, int64_t step, int32_t N, uint64_t se
     if (N < 1 || N > c->Nmax || N % c->world != 0 || step < 0) return fail(c, MPCGS_E_ARG, "step_local args");
     mpcgs_status st = enter(c);
     if (st) return st;
-    if ((st = step_local_launch(c, seed, step, N, false, 0))) return st;
+    if ((st = step_local_launch(c, seed, step, N))) return st;
     if ((st = leave(c))) return st;
     return check_status(c);
 }
@@ -886,7 +939,7 @@ mpcgs_status mpcgs_step_trace(mpcgs_ctx* c, int64_t step, int32_t N, int32_t K, 
     mpcgs_status st = enter(c);
     if (st) return st;
     CU(cudaMemsetAsync(c->s.counters + 2, 0, 8, c->work));
-    if ((st = step_local_launch(c, seed, step, N, false, 0))) return st;
+    if ((st = step_local_launch(c, seed, step, N))) return st;
     CU(launch_draw(c->s, seed, step, N, K, 0, 0, c->work));
     std::vector<double> rec((size_t)(N + 1) * REC);
     int32_t ci[16];
@@ -1065,6 +1118,7 @@ void mpcgs_free(mpcgs_ctx* c) {
     if (c->ev_a) cudaEventDestroy(c->ev_a);
     if (c->ev_b) cudaEventDestroy(c->ev_b);
     if (c->own_ws && c->ws) cudaFree(c->ws);
+    if (c->flush_buf) cudaFree(c->flush_buf);
     if (c->work) cudaStreamDestroy(c->work);
     delete c;
 }

@@ -224,9 +224,11 @@ template <typename T, int D>
 static cudaError_t launch_one(const PruneArgs& a, int ntrees, cudaStream_t st) {
     size_t smem = (size_t)a.nops * (sizeof(typename Traits<T>::E4) + sizeof(uint32_t));
     auto kern = k_prune<T, D>;
-    if (smem > 48 * 1024) {
+    static size_t attr_bytes = 48 * 1024;  // raised once, outside graph capture (first launch is at init)
+    if (smem > attr_bytes) {
         cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
         if (e != cudaSuccess) return e;
+        attr_bytes = smem;
     }
     dim3 grid(a.tiles, ntrees);
     kern<<<grid, PRUNE_THREADS, smem, st>>>(a);

@@ -271,9 +271,11 @@ size_t context_smem_bytes(int n) {
 
 cudaError_t launch_context(const DevState& s, uint64_t seed, int64_t step, cudaStream_t st) {
     size_t smem = context_smem_bytes(s.n);
-    if (smem > 48 * 1024) {
+    static size_t attr_bytes = 48 * 1024;
+    if (smem > attr_bytes) {
         cudaError_t e = cudaFuncSetAttribute(k_context, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
         if (e != cudaSuccess) return e;
+        attr_bytes = smem;
     }
     k_context<<<1, CTX_THREADS, smem, st>>>(s, seed, step);
     return cudaGetLastError();
