@@ -68,6 +68,7 @@ struct mpcgs_ctx {
     bool own_ws = false;
     double* score_out = nullptr;
     unsigned* theta_cnt = nullptr;
+    uint32_t* codes2 = nullptr;
     int64_t nsamples = 0;
     int lastN = 0;
     bool sticky = false;
@@ -108,13 +109,16 @@ mpcgs_status fail(mpcgs_ctx* c, mpcgs_status st, const std::string& msg) {
 
 // ------------------------------------------------------------ workspace layout
 struct Layout {
-    size_t codes, parent, left, right, need, age, e, em, gen, ctx_i, ctx_d, tau, len, lcnt, entry, omega, fixed;
+    size_t codes, codes2, parent, left, right, need, age, e, em, gen, ctx_i, ctx_d, tau, len, lcnt, entry, omega, fixed;
     size_t rec, sched_op, sched_e, tile_part, tile_cnt, sS, sL, sStep, sSlot, counters, last_draws, theta_buf,
         theta_cnt, score_out, total;
     int tiles_max;
 };
 
 size_t al(size_t x) { return (x + 255) & ~(size_t)255; }
+
+// 2-bit packed tip codes, 16 sites per 32-bit word, rows padded past the last tile
+int codes2_words(int L) { return ((L + 4096 + 63) / 64) * 4; }
 
 Layout layout(int n, int L, int Nmax, int64_t Mmax, int precision) {
     Layout y{};
@@ -129,6 +133,7 @@ Layout layout(int n, int L, int Nmax, int64_t Mmax, int precision) {
         return r;
     };
     y.codes = take((size_t)n * Lpad);
+    y.codes2 = take(4 * (size_t)n * codes2_words(L));
     y.parent = take(4 * (size_t)nn);
     y.left = take(4 * (size_t)nn);
     y.right = take(4 * (size_t)nn);
@@ -317,24 +322,31 @@ void upgma(int n, int L, const uint8_t* codes, double theta0, int32_t* parent, d
     }
 }
 
-// sites per CTA so that the pruning grid has enough CTAs (>= ~8 per SM)
-void prune_tiling(int L, int ntrees, int& tiles, int& sites_per_cta) {
-    long want = (long)148 * 8;
-    int spt = (int)std::max<long>(1, std::min<long>(16, ((long)ntrees * L) / (PRUNE_THREADS * want)));
-    sites_per_cta = spt * PRUNE_THREADS;
+// Sites per CTA: a multiple of the kernel's site batch, as many batches as keep
+// >= ~8 CTAs per SM busy.  Depends only on L and the GLOBAL tree count, so every
+// rank tiles (and sums) a proposal's sites identically (world-size invariance).
+void prune_tiling(int L, int ntrees_global, int precision, int& tiles, int& sites_per_cta) {
+    const int batch = prune_batch_sites(precision);
+    const long batches = (L + batch - 1) / batch;
+    const long want = (long)148 * 8;
+    const int per = (int)std::max<long>(1, std::min<long>(8, (ntrees_global * batches) / want));
+    sites_per_cta = per * batch;
     tiles = (L + sites_per_cta - 1) / sites_per_cta;
 }
 
-PruneArgs prune_args(mpcgs_ctx* c, int ntrees, double* out, int out_first, int out_stride) {
+PruneArgs prune_args(mpcgs_ctx* c, int ntrees_global, double* out, int out_first, int out_stride) {
     PruneArgs a{};
     a.codes = c->s.codes;
+    a.codes2 = c->codes2;
+    a.W2 = codes2_words(c->L);
     a.Lpad = c->Lpad;
     a.L = c->L;
     a.nops = c->nops;
     for (int i = 0; i < 4; ++i) a.pi[i] = c->s.pi[i];
     a.sched_op = c->s.sched_op;
     a.sched_e = c->s.sched_e;
-    prune_tiling(c->L, ntrees, a.tiles, a.sites_per_cta);
+    prune_tiling(c->L, ntrees_global, c->precision, a.tiles, a.sites_per_cta);
+    a.max_need = prune_max_need(c->n);
     a.tile_part = c->s.tile_part;
     a.tile_cnt = c->s.tile_cnt;
     a.out = out;
@@ -423,7 +435,7 @@ mpcgs_status step_local_launch(mpcgs_ctx* c, uint64_t seed, int64_t step, int N,
     int first = 1 + c->rank * (N / c->world), count = N / c->world;
     CU(launch_context(c->s, seed, step, c->work));
     CU(launch_propose(c->s, seed, step, first, count, c->work));
-    PruneArgs a = prune_args(c, count, c->s.rec, first, REC);
+    PruneArgs a = prune_args(c, N, c->s.rec, first, REC);
     if (pre) CU(cudaEventRecord(pre, c->work));
     CU(launch_prune(a, count, c->depth, c->precision, c->work));
     if (post) CU(cudaEventRecord(post, c->work));
@@ -694,11 +706,18 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
         s.Mmax = c->Mmax;
         c->theta_cnt = (unsigned*)(b + y.theta_cnt);
         c->score_out = (double*)(b + y.score_out);
+        c->codes2 = (uint32_t*)(b + y.codes2);
         if ((st = enter(c))) break;
         if (cudaMemsetAsync(c->ws, 0, y.total, c->work) != cudaSuccess) { st = fail(c, MPCGS_E_CUDA, "memset"); break; }
         std::vector<uint8_t> padded((size_t)n * c->Lpad, 0);
         for (int i = 0; i < n; ++i) std::memcpy(padded.data() + (size_t)i * c->Lpad, codes.data() + (size_t)i * L, L);
-        if (cudaMemcpyAsync((void*)s.codes, padded.data(), padded.size(), cudaMemcpyHostToDevice, c->work) != cudaSuccess) {
+        const int W2 = codes2_words(L);
+        std::vector<uint32_t> packed((size_t)n * W2, 0u);
+        for (int i = 0; i < n; ++i)
+            for (int site = 0; site < L; ++site)
+                packed[(size_t)i * W2 + (site >> 4)] |= (uint32_t)codes[(size_t)i * L + site] << (2 * (site & 15));
+        if (cudaMemcpyAsync((void*)s.codes, padded.data(), padded.size(), cudaMemcpyHostToDevice, c->work) != cudaSuccess ||
+            cudaMemcpyAsync(c->codes2, packed.data(), packed.size() * 4, cudaMemcpyHostToDevice, c->work) != cudaSuccess) {
             st = fail(c, MPCGS_E_CUDA, "codes upload");
             break;
         }

@@ -7,14 +7,19 @@
 namespace mpcgs {
 
 constexpr int PRUNE_THREADS = 128;
+constexpr int PRUNE_SI64 = 2;  // sites interleaved per thread, FP64 partials
+constexpr int PRUNE_SI32 = 2;  // FP32 partials
+constexpr int PRUNE_DR = 4;    // register-resident stack levels (deeper ones spill to shared memory)
 
 struct PruneArgs {
-    const uint8_t* codes;
-    int Lpad, L, nops;
+    const uint8_t* codes;       // [n][Lpad] bytes (flat kernel)
+    const uint32_t* codes2;     // [n][W2] 2-bit packed, 16 sites per word (table kernel)
+    int Lpad, L, nops, W2;
     double pi[4];
     const uint32_t* sched_op;  // [ntrees][nops]
     const void* sched_e;       // [ntrees][nops] float4 / double4
     int tiles, sites_per_cta;
+    int max_need;              // largest register need of any tree in the launch (<= floor(log2 n))
     double* tile_part;         // [ntrees][tiles]
     uint32_t* tile_cnt;        // [ntrees], zero on entry, reset by the kernel
     double* out;               // logL of tree t -> out[(out_first + t) * out_stride]
@@ -22,6 +27,9 @@ struct PruneArgs {
 };
 
 int prune_depth_for(int n);
+int prune_max_need(int n);
+int prune_batch_sites(int precision);      // sites_per_cta must be a multiple of this
+bool prune_uses_tables(int n, int precision);
 cudaError_t launch_prune(const PruneArgs& a, int ntrees, int depth, int precision, cudaStream_t st);
 
 // step kernels (step.cu); step < 0 -> read the step index from counters[0]

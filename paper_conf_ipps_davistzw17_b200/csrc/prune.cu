@@ -220,11 +220,440 @@ __global__ void __launch_bounds__(PRUNE_THREADS) k_prune(PruneArgs a) {
     }
 }
 
+// ============================================================================
+// Table kernel (the production path).  Tip codes are staged per site batch in
+// shared memory (2-bit packed, cp.async double buffer); every tip child reads
+// its 4-vector P_{.,x}(t) from a per-op 4x4 table and every cherry (two tip
+// children) its product vector from a 16x4 table, both built in shared memory
+// at CTA start; SI sites per thread are interleaved so that one dispatch and one
+// read of the op serve SI register stacks.  The register stack holds DR levels;
+// deeper levels (rare: need > DR) live in shared memory, so one compiled kernel
+// scores every tree shape.
+// ============================================================================
+__device__ __forceinline__ void cp_async16(void* smem, const void* gmem) {
+    unsigned sa = (unsigned)__cvta_generic_to_shared(smem);
+    asm volatile("cp.async.cg.shared.global [%0], [%1], 16;\n" ::"r"(sa), "l"(gmem));
+}
+__device__ __forceinline__ void cp_async_commit() { asm volatile("cp.async.commit_group;\n" ::); }
+template <int N>
+__device__ __forceinline__ void cp_async_wait() { asm volatile("cp.async.wait_group %0;\n" ::"n"(N)); }
+
+template <typename T>
+__device__ __forceinline__ void ld4(T (&r)[4], const T* p);
+template <>
+__device__ __forceinline__ void ld4<double>(double (&r)[4], const double* p) {
+    const double2 a = reinterpret_cast<const double2*>(p)[0];
+    const double2 b = reinterpret_cast<const double2*>(p)[1];
+    r[0] = a.x; r[1] = a.y; r[2] = b.x; r[3] = b.y;
+}
+template <>
+__device__ __forceinline__ void ld4<float>(float (&r)[4], const float* p) {
+    const float4 a = *reinterpret_cast<const float4*>(p);
+    r[0] = a.x; r[1] = a.y; r[2] = a.z; r[3] = a.w;
+}
+
+template <typename T>
+__device__ __forceinline__ T pick4(const T (&v)[4], int x) {
+    return x == 0 ? v[0] : (x == 1 ? v[1] : (x == 2 ? v[2] : v[3]));
+}
+
+// exponent test of one 4-vector: k > 0 if max < 2^-TS (then max * 2^k in [1, 2))
+__device__ __forceinline__ int rescale_k(const double (&r)[4]) {
+    const int m = max(max(hi_bits(r[0]), hi_bits(r[1])), max(hi_bits(r[2]), hi_bits(r[3])));
+    return m < ((1023 - Traits<double>::TS) << 20) ? min(1023 - (m >> 20), 1000) : 0;
+}
+__device__ __forceinline__ int rescale_k(const float (&r)[4]) {
+    const int m = max(max(hi_bits(r[0]), hi_bits(r[1])), max(hi_bits(r[2]), hi_bits(r[3])));
+    return m < ((127 - Traits<float>::TS) << 23) ? min(127 - (m >> 23), 120) : 0;
+}
+__device__ __forceinline__ double pow2(int k, double) { return __hiloint2double((1023 + k) << 20, 0); }
+__device__ __forceinline__ float pow2(int k, float) { return __int_as_float((127 + k) << 23); }
+
+// Rescale when any site of any lane has max < 2^-TS: the per-site test is
+// cheap (integer max of the high words); the multiply is a rare warp-uniform branch.
+__device__ __forceinline__ bool small4(const double (&r)[4]) {
+    const int m = max(max(hi_bits(r[0]), hi_bits(r[1])), max(hi_bits(r[2]), hi_bits(r[3])));
+    return m < ((1023 - Traits<double>::TS) << 20);
+}
+__device__ __forceinline__ bool small4(const float (&r)[4]) {
+    const int m = max(max(hi_bits(r[0]), hi_bits(r[1])), max(hi_bits(r[2]), hi_bits(r[3])));
+    return m < ((127 - Traits<float>::TS) << 23);
+}
+template <typename T, int SI>
+__device__ __forceinline__ void rescale_sites(T (&v)[SI][4], int (&scale)[SI]) {
+    bool any = false;
+#pragma unroll
+    for (int q = 0; q < SI; ++q) any |= small4(v[q]);
+    if (__any_sync(0xffffffffu, any)) {
+#pragma unroll
+        for (int q = 0; q < SI; ++q) {
+            const int k = rescale_k(v[q]);
+            const T f = pow2(k, T(0));
+            v[q][0] *= f; v[q][1] *= f; v[q][2] *= f; v[q][3] *= f;
+            scale[q] += k;
+        }
+    }
+}
+
+// Register stack of DR levels per site, deeper levels in shared memory laid out
+// [level][site k][state X][thread] (conflict-free).
+template <typename T, int DR, int SI>
+struct Stack {
+    T r[SI][DR][4];
+    T* sm;  // this thread's column of the spill area
+    template <int S>
+    __device__ __forceinline__ void get(int k, T (&v)[4]) const {
+        if constexpr (S < DR) {
+            v[0] = r[k][S][0]; v[1] = r[k][S][1]; v[2] = r[k][S][2]; v[3] = r[k][S][3];
+        } else {
+#pragma unroll
+            for (int x = 0; x < 4; ++x) v[x] = sm[(((S - DR) * SI + k) * 4 + x) * PRUNE_THREADS];
+        }
+    }
+    template <int S>
+    __device__ __forceinline__ void put(int k, const T (&v)[4]) {
+        if constexpr (S < DR) {
+            r[k][S][0] = v[0]; r[k][S][1] = v[1]; r[k][S][2] = v[2]; r[k][S][3] = v[3];
+        } else {
+#pragma unroll
+            for (int x = 0; x < 4; ++x) sm[(((S - DR) * SI + k) * 4 + x) * PRUNE_THREADS] = v[x];
+        }
+    }
+};
+
+// Tip codes of the current site batch in shared memory, 2-bit packed (16 sites
+// per 32-bit word, a thread's SI sites adjacent).  The byte offset of a site's
+// table entry is one funnel rotation and one mask: rotating the word right by
+// (bit position - log2(entry bytes)) puts the 2-bit code at the entry-size bit.
+template <bool CB, int SI>
+struct Codes {
+    static_assert(!CB, "byte codes retired");
+    const unsigned char* base;  // this batch's buffer
+    int wofs;                   // word index of this thread's sites
+    uint32_t rb[SI], ra[SI];    // rotations for the code * EB and code * 4 * EB offsets
+    static constexpr int BATCH = PRUNE_THREADS * SI;
+    static constexpr int WB = BATCH / 16;
+    template <int EB>
+    __device__ __forceinline__ void init(int tid) {
+        constexpr int LG = EB == 32 ? 5 : 4;
+        wofs = (tid * SI) >> 4;
+#pragma unroll
+        for (int k = 0; k < SI; ++k) {
+            const int p = ((tid * SI) & 15) * 2 + 2 * k;  // bit position of site k's code
+            rb[k] = (uint32_t)(p - LG) & 31u;
+            ra[k] = (uint32_t)(p - LG - 2) & 31u;
+        }
+    }
+    __device__ __forceinline__ uint32_t word(int tip) const {
+        return reinterpret_cast<const uint32_t*>(base)[tip * WB + wofs];
+    }
+    template <int EB>
+    __device__ __forceinline__ uint32_t off(uint32_t w, int k) const {  // code * EB
+        return __funnelshift_r(w, w, rb[k]) & (3u * EB);
+    }
+    template <int EB>
+    __device__ __forceinline__ uint32_t off4(uint32_t w, int k) const {  // code * 4 * EB
+        return __funnelshift_r(w, w, ra[k]) & (12u * EB);
+    }
+    static constexpr size_t buf_bytes(int n) { return (size_t)n * WB * 4; }
+};
+
+constexpr uint32_t TAB_CHECK = 0x80000000u;  // toff flag: the cherry table can hold small vectors
+
+template <typename T, int DR, int SI, bool CB, int S, int DMX>
+__device__ __forceinline__ void tab_tt(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, const T* s_tab,
+                                       const Codes<CB, SI>& c, int (&scale)[SI]) {
+    if constexpr (S < DMX) {
+        constexpr int EB = 4 * sizeof(T);
+        const uint32_t wa = c.word((code >> 6) & 2047);
+        const uint32_t wb = c.word((code >> 17) & 2047);
+        const char* base = reinterpret_cast<const char*>(s_tab) + (toff & ~TAB_CHECK);
+        T v[SI][4];
+#pragma unroll
+        for (int k = 0; k < SI; ++k)
+            ld4<T>(v[k], reinterpret_cast<const T*>(base + c.template off4<EB>(wa, k) + c.template off<EB>(wb, k)));
+        if (toff & TAB_CHECK) rescale_sites<T, SI>(v, scale);
+#pragma unroll
+        for (int k = 0; k < SI; ++k) st.template put<S>(k, v[k]);
+    }
+}
+
+template <typename T, int DR, int SI, bool CB, int S, int DMX>
+__device__ __forceinline__ void tab_ts(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff,
+                                       const typename Traits<T>::E4& ed, const T* s_tab, const Codes<CB, SI>& c,
+                                       const T (&pi)[4], int (&scale)[SI]) {
+    if constexpr (S >= 1 && S <= DMX) {
+        constexpr int EB = 4 * sizeof(T);
+        const uint32_t wa = c.word((code >> 6) & 2047);
+        const char* base = reinterpret_cast<const char*>(s_tab) + toff;
+        T v[SI][4];
+#pragma unroll
+        for (int k = 0; k < SI; ++k) {
+            T tip[4];
+            ld4<T>(tip, reinterpret_cast<const T*>(base + c.template off<EB>(wa, k)));
+            st.template get<S - 1>(k, v[k]);
+            branch<T>(v[k], ed.z, ed.w, pi);
+#pragma unroll
+            for (int i = 0; i < 4; ++i) v[k][i] *= tip[i];
+        }
+        rescale_sites<T, SI>(v, scale);
+#pragma unroll
+        for (int k = 0; k < SI; ++k) st.template put<S - 1>(k, v[k]);
+    }
+}
+
+template <typename T, int DR, int SI, int S, int DMX>
+__device__ __forceinline__ void tab_ss(Stack<T, DR, SI>& st, const typename Traits<T>::E4& ed, const T (&pi)[4],
+                                       int (&scale)[SI]) {
+    if constexpr (S >= 2 && S <= DMX) {
+        T v[SI][4];
+#pragma unroll
+        for (int k = 0; k < SI; ++k) {
+            T w[4];
+            st.template get<S - 2>(k, v[k]);
+            st.template get<S - 1>(k, w);
+            branch<T>(v[k], ed.x, ed.y, pi);
+            branch<T>(w, ed.z, ed.w, pi);
+#pragma unroll
+            for (int i = 0; i < 4; ++i) v[k][i] *= w[i];
+        }
+        rescale_sites<T, SI>(v, scale);
+#pragma unroll
+        for (int k = 0; k < SI; ++k) st.template put<S - 2>(k, v[k]);
+    }
+}
+
+#define MPCGS_TABCASE(S)                                                                          \
+    case 3 * (S) + 0: tab_tt<T, DR, SI, CB, S, DMX>(st, code, toff, s_tab, cc, scale); break;       \
+    case 3 * (S) + 1: tab_ts<T, DR, SI, CB, S, DMX>(st, code, toff, ed, s_tab, cc, pi, scale); break; \
+    case 3 * (S) + 2: tab_ss<T, DR, SI, S, DMX>(st, ed, pi, scale); break;
+#define MPCGS_CASES_4 MPCGS_TABCASE(0) MPCGS_TABCASE(1) MPCGS_TABCASE(2) MPCGS_TABCASE(3) MPCGS_TABCASE(4)
+#define MPCGS_CASES_6 MPCGS_CASES_4 MPCGS_TABCASE(5) MPCGS_TABCASE(6)
+#define MPCGS_CASES_8 MPCGS_CASES_6 MPCGS_TABCASE(7) MPCGS_TABCASE(8)
+#define MPCGS_CASES_10 MPCGS_CASES_8 MPCGS_TABCASE(9) MPCGS_TABCASE(10)
+
+// one op for SI sites; the switch only has the (sp, type) labels a DMX-level tree can use
+template <typename T, int DR, int SI, bool CB, int DMX>
+__device__ __forceinline__ void run_op(int di, Stack<T, DR, SI>& st, uint32_t code, uint32_t toff,
+                                       const typename Traits<T>::E4& ed, const T* s_tab, const Codes<CB, SI>& cc,
+                                       const T (&pi)[4], int (&scale)[SI]) {
+    if constexpr (DMX <= 4) {
+        switch (di) { MPCGS_CASES_4 default: break; }
+    } else if constexpr (DMX <= 6) {
+        switch (di) { MPCGS_CASES_6 default: break; }
+    } else if constexpr (DMX <= 8) {
+        switch (di) { MPCGS_CASES_8 default: break; }
+    } else {
+        switch (di) { MPCGS_CASES_10 default: break; }
+    }
+}
+
+__host__ __device__ constexpr size_t align16(size_t x) { return (x + 15) & ~(size_t)15; }
+
+// shared memory of the table kernel for trees of n tips whose register need is
+// at most `need` (spill levels above DR)
+template <typename T, int DR, int SI, bool CB>
+__host__ __device__ size_t tab_smem_bytes(int nops, int need) {
+    const int n = nops + 1;
+    const int spill = need > DR ? need - DR : 0;
+    return align16(sizeof(typename Traits<T>::E4) * nops) + align16(sizeof(T) * 32 * (size_t)n) +
+           align16(sizeof(uint2) * nops) + 2 * align16(Codes<CB, SI>::buf_bytes(n)) +
+           sizeof(T) * (size_t)spill * SI * 4 * PRUNE_THREADS;
+}
+
+template <typename T, int DR, int SI, bool CB, int DMX>
+__global__ void __launch_bounds__(PRUNE_THREADS) k_prune_tab(PruneArgs a) {
+    using E4 = typename Traits<T>::E4;
+    using CD = Codes<CB, SI>;
+    constexpr int BATCH = CD::BATCH;  // sites per batch
+    extern __shared__ __align__(16) unsigned char smem_raw[];
+    const int nops = a.nops, n = nops + 1;
+    E4* s_e = reinterpret_cast<E4*>(smem_raw);
+    T* s_tab = reinterpret_cast<T*>(smem_raw + align16(sizeof(E4) * nops));
+    uint2* s_op = reinterpret_cast<uint2*>(reinterpret_cast<unsigned char*>(s_tab) + align16(sizeof(T) * 32 * n));
+    unsigned char* s_cod = reinterpret_cast<unsigned char*>(s_op) + align16(sizeof(uint2) * nops);
+    const size_t bufb = align16(CD::buf_bytes(n));
+    T* s_spill = reinterpret_cast<T*>(s_cod + 2 * bufb);
+    __shared__ double s_red[PRUNE_THREADS / 32];
+    __shared__ bool s_last;
+
+    const int tid = threadIdx.x;
+    const int tree = blockIdx.y;
+    const int tile = blockIdx.x;
+    const int s_begin = tile * a.sites_per_cta;
+    const int s_end = min(a.L, s_begin + a.sites_per_cta);
+    const int nb = (s_end - s_begin + BATCH - 1) / BATCH;
+
+    auto issue = [&](int b, int buf) {
+        const int site0 = s_begin + b * BATCH;
+        unsigned char* dst = s_cod + (size_t)buf * bufb;
+        constexpr int WB = CD::WB, CH = WB / 4;  // 16-byte chunks per tip row
+        const uint32_t* src = a.codes2 + (site0 >> 4);
+        for (int c = tid; c < n * CH; c += PRUNE_THREADS) {
+            const int tip = c / CH, q = c - tip * CH;
+            cp_async16(dst + ((size_t)tip * WB + q * 4) * 4, src + (size_t)tip * a.W2 + q * 4);
+        }
+        cp_async_commit();
+    };
+    if (nb > 0) issue(0, 0);
+
+    // schedule, then per-op table byte offsets (warp 0 scan), then the tables
+    const uint32_t* __restrict__ gop = a.sched_op + (size_t)tree * nops;
+    const E4* __restrict__ ge = reinterpret_cast<const E4*>(a.sched_e) + (size_t)tree * nops;
+    for (int i = tid; i < nops; i += PRUNE_THREADS) {
+        s_op[i].x = gop[i];
+        s_e[i] = ge[i];
+    }
+    __syncthreads();
+    if (tid < 32) {
+        uint32_t carry = 0;
+        for (int base = 0; base < nops; base += 32) {
+            const int i = base + tid;
+            uint32_t sz = 0;
+            if (i < nops) {
+                const uint32_t ty = s_op[i].x & 3u;
+                sz = ty == OP_TT ? 64u : (ty == OP_TS ? 16u : 0u);
+            }
+            uint32_t x = sz;
+#pragma unroll
+            for (int o = 1; o < 32; o <<= 1) {
+                const uint32_t y = __shfl_up_sync(0xffffffffu, x, o);
+                if (tid >= o) x += y;
+            }
+            if (i < nops) s_op[i].y = (carry + x - sz) * (uint32_t)sizeof(T);  // byte offset
+            carry += __shfl_sync(0xffffffffu, x, 31);
+        }
+    }
+    __syncthreads();
+    const T pi[4] = {(T)a.pi[0], (T)a.pi[1], (T)a.pi[2], (T)a.pi[3]};
+    for (int idx = tid; idx < nops * 64; idx += PRUNE_THREADS) {
+        const int op = idx >> 6, j = idx & 63;
+        const uint32_t ty = s_op[op].x & 3u;
+        T* tab = reinterpret_cast<T*>(reinterpret_cast<char*>(s_tab) + s_op[op].y);
+        const E4 ed = s_e[op];
+        if (ty == OP_TT) {
+            // cherry: entry (xa, xb) = P_{.,xa}(t_a) (.) P_{.,xb}(t_b)   (Eq. 19-20 at two tips)
+            const int xa = j >> 4, xb = (j >> 2) & 3, X = j & 3;
+            const T va = (X == xa ? (T)ed.x : T(0)) + (T)ed.y * pick4(pi, xa);
+            const T vb = (X == xb ? (T)ed.z : T(0)) + (T)ed.w * pick4(pi, xb);
+            tab[j] = va * vb;
+        } else if (ty == OP_TS && j < 16) {
+            const int x = j >> 2, X = j & 3;
+            tab[j] = (X == x ? (T)ed.x : T(0)) + (T)ed.y * pick4(pi, x);
+        }
+    }
+    __syncthreads();
+    // flag cherry tables with an entry whose max is below the rescale threshold
+    for (int op = tid; op < nops; op += PRUNE_THREADS) {
+        if ((s_op[op].x & 3u) != OP_TT) continue;
+        const T* tab = reinterpret_cast<const T*>(reinterpret_cast<const char*>(s_tab) + s_op[op].y);
+        bool small = false;
+        for (int e = 0; e < 16; ++e) {
+            T v[4];
+            ld4<T>(v, tab + 4 * e);
+            small |= small4(v);
+        }
+        if (small) s_op[op].y |= TAB_CHECK;
+    }
+
+    double mant = 1.0;
+    int expo = 0;
+    Stack<T, DR, SI> st;
+    st.sm = s_spill + tid;
+#pragma unroll
+    for (int k = 0; k < SI; ++k)
+#pragma unroll
+        for (int i = 0; i < DR; ++i)
+#pragma unroll
+            for (int j = 0; j < 4; ++j) st.r[k][i][j] = T(0);
+
+    CD cc;
+    cc.template init<4 * sizeof(T)>(tid);
+    for (int b = 0; b < nb; ++b) {
+        if (b + 1 < nb) {
+            issue(b + 1, (b + 1) & 1);
+            cp_async_wait<1>();
+        } else {
+            cp_async_wait<0>();
+        }
+        __syncthreads();
+        cc.base = s_cod + (size_t)(b & 1) * bufb;
+        int scale[SI];
+#pragma unroll
+        for (int k = 0; k < SI; ++k) scale[k] = 0;
+        for (int op = 0; op < nops; ++op) {
+            const uint2 ox = s_op[op];
+            const E4 ed = s_e[op];
+            const int di = (int)((ox.x >> 2) & 15u) * 3 + (int)(ox.x & 3u);  // dense (sp, type) index
+            run_op<T, DR, SI, CB, DMX>(di, st, ox.x, ox.y, ed, s_tab, cc, pi, scale);
+        }
+        const int site0 = s_begin + b * BATCH + tid * SI;
+#pragma unroll
+        for (int k = 0; k < SI; ++k) {
+            T root[4];
+            st.template get<0>(k, root);
+            T ls = pi[0] * root[0];   // Eq. 21
+            ls = fma(pi[1], root[1], ls);
+            ls = fma(pi[2], root[2], ls);
+            ls = fma(pi[3], root[3], ls);
+            if (site0 + k < s_end) {  // sites past L (padding) are computed, not counted
+                mant *= (double)ls;
+                const int hi = __double2hiint(mant);
+                const int ex = ((hi >> 20) & 2047) - 1023;
+                if (ex > -1023) {
+                    mant = __hiloint2double((hi & 0x800FFFFF) | (1023 << 20), __double2loint(mant));
+                    expo += ex;
+                }
+                expo -= scale[k];
+            }
+        }
+        __syncthreads();  // the buffer of batch b is refilled in iteration b+1
+    }
+    double ll = (mant > 0.0) ? log(mant) + (double)expo * 0.69314718055994530942 : -INFINITY;
+
+#pragma unroll
+    for (int off = 16; off > 0; off >>= 1) ll += __shfl_down_sync(0xffffffffu, ll, off);
+    if ((tid & 31) == 0) s_red[tid >> 5] = ll;
+    __syncthreads();
+    if (tid == 0) {
+        double t = 0.0;
+        for (int w = 0; w < PRUNE_THREADS / 32; ++w) t += s_red[w];
+        a.tile_part[(size_t)tree * a.tiles + tile] = t;
+        __threadfence();
+        const unsigned prev = atomicAdd(a.tile_cnt + tree, 1u);
+        s_last = (prev == (unsigned)(a.tiles - 1));
+    }
+    __syncthreads();
+    if (s_last && tid == 0) {
+        __threadfence();
+        double t = 0.0;
+        const volatile double* tp = a.tile_part + (size_t)tree * a.tiles;
+        for (int k = 0; k < a.tiles; ++k) t += tp[k];
+        a.out[(size_t)(a.out_first + tree) * a.out_stride] = t;
+        a.tile_cnt[tree] = 0u;
+    }
+}
+
 template <typename T, int D>
-static cudaError_t launch_one(const PruneArgs& a, int ntrees, cudaStream_t st) {
+static cudaError_t launch_flat(const PruneArgs& a, int ntrees, cudaStream_t st) {
     size_t smem = (size_t)a.nops * (sizeof(typename Traits<T>::E4) + sizeof(uint32_t));
     auto kern = k_prune<T, D>;
     static size_t attr_bytes = 48 * 1024;  // raised once, outside graph capture (first launch is at init)
+    if (smem > attr_bytes) {
+        cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+        if (e != cudaSuccess) return e;
+        attr_bytes = smem;
+    }
+    dim3 grid(a.tiles, ntrees);
+    kern<<<grid, PRUNE_THREADS, smem, st>>>(a);
+    return cudaGetLastError();
+}
+
+template <typename T, int DR, int SI, bool CB, int DMX>
+static cudaError_t launch_tab(const PruneArgs& a, int ntrees, cudaStream_t st) {
+    const size_t smem = tab_smem_bytes<T, DR, SI, CB>(a.nops, a.max_need);
+    auto kern = k_prune_tab<T, DR, SI, CB, DMX>;
+    static size_t attr_bytes = 48 * 1024;
     if (smem > attr_bytes) {
         cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
         if (e != cudaSuccess) return e;
@@ -244,22 +673,49 @@ int prune_depth_for(int n) {
     return 10;
 }
 
+int prune_max_need(int n) {
+    int d = 0;
+    while ((2 << d) <= n) ++d;
+    return d < 1 ? 1 : d;
+}
+
+int prune_batch_sites(int precision) { return PRUNE_THREADS * (precision == 32 ? PRUNE_SI32 : PRUNE_SI64); }
+
+bool prune_code_bytes(int, int) { return false; }
+
+bool prune_uses_tables(int n, int precision) {
+    const int need = prune_max_need(n);
+    const size_t bytes = precision == 32 ? tab_smem_bytes<float, PRUNE_DR, PRUNE_SI32, false>(n - 1, need)
+                                         : tab_smem_bytes<double, PRUNE_DR, PRUNE_SI64, false>(n - 1, need);
+    return bytes <= 160 * 1024;
+}
+
+template <typename T, int SI, bool CB>
+static cudaError_t launch_tab_dmx(const PruneArgs& a, int ntrees, int depth, cudaStream_t st) {
+    switch (depth) {
+        case 4: return launch_tab<T, PRUNE_DR, SI, CB, 4>(a, ntrees, st);
+        case 6: return launch_tab<T, PRUNE_DR, SI, CB, 6>(a, ntrees, st);
+        case 8: return launch_tab<T, PRUNE_DR, SI, CB, 8>(a, ntrees, st);
+        default: return launch_tab<T, PRUNE_DR, SI, CB, 10>(a, ntrees, st);
+    }
+}
+
+template <typename T, int SI>
+static cudaError_t launch_typed(const PruneArgs& a, int ntrees, int depth, bool tab, cudaStream_t st) {
+    if (tab) return launch_tab_dmx<T, SI, false>(a, ntrees, depth, st);
+    switch (depth) {
+        case 4: return launch_flat<T, 4>(a, ntrees, st);
+        case 6: return launch_flat<T, 6>(a, ntrees, st);
+        case 8: return launch_flat<T, 8>(a, ntrees, st);
+        default: return launch_flat<T, 10>(a, ntrees, st);
+    }
+}
+
 cudaError_t launch_prune(const PruneArgs& a, int ntrees, int depth, int precision, cudaStream_t st) {
     if (ntrees <= 0) return cudaSuccess;
-    if (precision == 32) {
-        switch (depth) {
-            case 4: return launch_one<float, 4>(a, ntrees, st);
-            case 6: return launch_one<float, 6>(a, ntrees, st);
-            case 8: return launch_one<float, 8>(a, ntrees, st);
-            default: return launch_one<float, 10>(a, ntrees, st);
-        }
-    }
-    switch (depth) {
-        case 4: return launch_one<double, 4>(a, ntrees, st);
-        case 6: return launch_one<double, 6>(a, ntrees, st);
-        case 8: return launch_one<double, 8>(a, ntrees, st);
-        default: return launch_one<double, 10>(a, ntrees, st);
-    }
+    const bool tab = a.codes2 != nullptr && prune_uses_tables(a.nops + 1, precision);
+    if (precision == 32) return launch_typed<float, PRUNE_SI32>(a, ntrees, depth, tab, st);
+    return launch_typed<double, PRUNE_SI64>(a, ntrees, depth, tab, st);
 }
 
 }  // namespace mpcgs
