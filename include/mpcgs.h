@@ -77,7 +77,9 @@ typedef struct {
     const double* init_age;     /* host [2n-1]; used with init_parent */
     int32_t rank, world;   /* world = 1: one GPU.  world > 1: proposals sharded over ranks */
     const void* nccl_id;   /* host, 128 bytes: ncclUniqueId made by rank 0 with
-                              mpcgs_nccl_unique_id() and broadcast by the caller; NULL if world = 1 */
+                              mpcgs_nccl_unique_id() and broadcast by the caller.  NULL with
+                              world > 1: no communicator; the caller exchanges records itself
+                              (mpcgs_step_local / get_records / put_records / step_finish) */
     void* stream;          /* cudaStream_t for all work; NULL = the legacy default stream */
     void* workspace;       /* device memory of >= mpcgs_workspace_bytes(...) bytes, 256-B aligned;
                               NULL -> the context allocates (and frees) its own */
@@ -94,7 +96,9 @@ size_t mpcgs_workspace_bytes(int32_t n_seq, int32_t n_sites, int32_t max_proposa
 
 /* Create a context: validate and copy the alignment, compute pi and u, build G0
  * (init_parent/init_age, else UPGMA), upload everything to the device and score
- * P(D|G0) with the pruning kernel.  theta0 > 0 is the driving value (L1239-1241). */
+ * P(D|G0) with the pruning kernel.  theta0 > 0 is the driving value (L1239-1241).
+ * On an error after allocation *out still receives the context so that
+ * mpcgs_last_error() can explain; the caller must mpcgs_free() it. */
 mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, double theta0,
                         mpcgs_ctx** out);
 

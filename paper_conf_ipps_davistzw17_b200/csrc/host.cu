@@ -722,9 +722,9 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
             break;
         }
         if ((st = upload_state(c, parent.data(), age.data()))) break;
-        if (c->world > 1) {
+        if (c->world > 1 && cfg->nccl_id) {  // without an id: host-staged record exchange only
             NcclApi& api = nccl();
-            if (!api.ok || !cfg->nccl_id) { st = fail(c, MPCGS_E_NCCL, "NCCL unavailable or nccl_id missing"); break; }
+            if (!api.ok) { st = fail(c, MPCGS_E_NCCL, "NCCL (libnccl.so.2) could not be loaded"); break; }
             ncclUniqueId id;
             std::memcpy(&id, cfg->nccl_id, sizeof(id));
             ncclResult_t r = api.commInitRank(&c->comm, c->world, id, c->rank);
@@ -767,6 +767,9 @@ mpcgs_status mpcgs_sample(mpcgs_ctx* c, int32_t N, int64_t M, uint64_t seed) {
     CHECK_CTX(c);
     if (N < 1 || N > c->Nmax || N % c->world != 0 || M < 0 || M > c->Mmax)
         return fail(c, MPCGS_E_ARG, "n_proposals / n_samples out of range or not divisible by world");
+    if (c->world > 1 && !c->comm)
+        return fail(c, MPCGS_E_STATE, "world > 1 without an NCCL id: drive steps with mpcgs_step_local, "
+                                      "mpcgs_get_records/put_records and mpcgs_step_finish");
     const int64_t steps = (int64_t)c->burnin + (M + N - 1) / N;
     mpcgs_status st = enter(c);
     if (st) return st;

@@ -304,18 +304,24 @@ __device__ void place_two(double len, double A, double B, double u1, double u2, 
     }
     const double target = u1 * two_cdf(len, len, A, B);
     double lo = 0.0, hi = len;
-    x = 0.5 * len;
-    for (int it = 0; it < 100; ++it) {
+    // start from the root of the dominant term (exact when e^{-B len} -> 0); the
+    // safeguarded iteration then converges to the same root as from len/2 (S13)
+    x = -log1p(-u1 * (-expm1(-(A + B) * len))) / (A + B);
+    if (!(x > 0.0 && x < len)) x = 0.5 * len;
+    // Newton to |dx| <= 2e-14 len (the closed-form CDF cancels when (A+B) len << 1,
+    // which bounds its attainable precision), at most 60 iterations
+    for (int it = 0; it < 60; ++it) {
         const double f = two_cdf(x, len, A, B) - target;
         const double d = exp(-(A + B) * x) - exp(-B * len - A * x);
+        if (f == 0.0) break;
         if (f > 0.0) hi = x;
         else lo = x;
         double xn = (d > 0.0) ? x - f / d : 0.5 * (lo + hi);
-        if (!(xn > lo && xn < hi)) xn = 0.5 * (lo + hi);
-        if (fabs(xn - x) <= 1e-15 * len) {
+        if (fabs(xn - x) <= 2e-14 * len) {  // converged Newton step (checked before the safeguard)
             x = xn;
             break;
         }
+        if (!(xn > lo && xn < hi)) xn = 0.5 * (lo + hi);
         x = xn;
     }
     y = x - log1p(u2 * expm1(-B * (len - x))) / B;
@@ -330,7 +336,13 @@ struct Walk {
 // Forward walk over the feasible intervals, young -> old (L1028-1034); RNG order
 // per interval: choice, event times, then the pair if the first coalescence
 // happens with three active lineages.
-__device__ Walk forward_walk(const DevState& s, int m, int k0, bool rootcase, uint64_t seed, uint32_t slot,
+struct WalkCtx {  // the step's interval context, staged in shared memory
+    const double *tau, *len, *omega;
+    const int *lcnt, *entry;
+    double theta0;
+};
+
+__device__ Walk forward_walk(const WalkCtx& s, int m, int k0, bool rootcase, uint64_t seed, uint32_t slot,
                              uint32_t step) {
     UStream us(seed, slot, step, TAG_PROPOSE);
     Walk w{0.0, 0.0, 0, 0};
@@ -400,6 +412,11 @@ __global__ void __launch_bounds__(32) k_propose(DevState s, uint64_t seed, int64
     int* sR = sL + nint;       // [n-1]
     int* sNeed = sR + nint;    // [nn]
     int* sStack = sNeed + nn;  // [2n]
+    int* sLc = sStack + 2 * n;  // [n+1] inactive counts
+    int* sEn = sLc + n + 1;     // [n+2] entry flags
+    double* sTau = reinterpret_cast<double*>(psm + ((4 * n + 2 + 4 * n) & ~1) + 4);  // [n+2]
+    double* sLen = sTau + n + 2;   // [n+1]
+    double* sOm = sLen + n + 1;    // [9(n+1)]
     __shared__ double sh_d[8];  // t1, t2, e/em of changed branches
     __shared__ int sh_i[8];
     const int lane = threadIdx.x;
@@ -413,8 +430,20 @@ __global__ void __launch_bounds__(32) k_propose(DevState s, uint64_t seed, int64
     const int c0 = s.ctx_i[6], c1 = s.ctx_i[7], c2 = s.ctx_i[8];
     const int nfixed = s.ctx_i[9], root = s.ctx_i[10];
 
+    // stage the interval context (L2 reads once, coalesced) for lane 0's sequential walk
+    for (int i = lane; i <= m; i += 32) {
+        sTau[i] = s.tau[i];
+        sEn[i] = s.entry[i];
+        if (i < m) {
+            sLen[i] = s.len[i];
+            sLc[i] = s.lcnt[i];
+        }
+    }
+    for (int i = lane; i < 9 * m; i += 32) sOm[i] = s.omega[i];
+    __syncwarp();
     if (lane == 0) {
-        Walk w = forward_walk(s, m, k0, rootcase, seed, (uint32_t)slot, (uint32_t)step);
+        const WalkCtx wc{sTau, sLen, sOm, sLc, sEn, s.theta0};
+        Walk w = forward_walk(wc, m, k0, rootcase, seed, (uint32_t)slot, (uint32_t)step);
         int pair = w.pair;
         double t1 = w.t1, t2 = w.t2;
         if (!w.ok) {
@@ -526,16 +555,30 @@ __global__ void __launch_bounds__(32) k_propose(DevState s, uint64_t seed, int64
     }
 }
 
-size_t propose_smem_bytes(int n) { return sizeof(int) * ((size_t)2 * (n - 1) + (2 * n - 1) + 2 * n); }
+size_t propose_smem_bytes(int n) {
+    return sizeof(int) * ((size_t)((4 * n + 2 + 4 * n) & ~1) + 4) + sizeof(double) * ((size_t)(n + 2) + (n + 1) + 9 * (n + 1));
+}
 
 cudaError_t launch_propose(const DevState& s, uint64_t seed, int64_t step, int slot_first, int count,
                            cudaStream_t st) {
     if (count <= 0) return cudaSuccess;
-    size_t smem = propose_smem_bytes(s.n);
-    if (s.precision == 32)
+    const size_t smem = propose_smem_bytes(s.n);
+    static size_t attr64 = 48 * 1024, attr32 = 48 * 1024;
+    if (s.precision == 32) {
+        if (smem > attr32) {
+            cudaError_t e = cudaFuncSetAttribute(k_propose<float4, float>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+            if (e != cudaSuccess) return e;
+            attr32 = smem;
+        }
         k_propose<float4, float><<<count, 32, smem, st>>>(s, seed, step, slot_first);
-    else
+    } else {
+        if (smem > attr64) {
+            cudaError_t e = cudaFuncSetAttribute(k_propose<double4, double>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+            if (e != cudaSuccess) return e;
+            attr64 = smem;
+        }
         k_propose<double4, double><<<count, 32, smem, st>>>(s, seed, step, slot_first);
+    }
     return cudaGetLastError();
 }
 

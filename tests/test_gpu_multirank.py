@@ -1,0 +1,58 @@
+"""World-size invariance on one GPU: P virtual ranks, each a
+context with (rank, world = P) scoring only its slots, exchange records
+through the C ABI (mpcgs_get_records / mpcgs_put_records) and draw with
+mpcgs_step_finish.  Every rank must reproduce the world = 1 chain bit for bit:
+same records, same draws, same generator."""
+import numpy as np
+import pytest
+
+import synth
+
+pytestmark = pytest.mark.gpu
+
+
+@pytest.fixture(scope="module")
+def P():
+    import torch
+
+    if not torch.cuda.is_available():
+        pytest.skip("no CUDA device")
+    import paper_conf_ipps_davistzw17_b200 as pkg
+
+    pkg.lib()
+    return pkg
+
+
+@pytest.mark.parametrize("world", [2, 4, 8])
+@pytest.mark.parametrize("precision", [64, 32])
+def test_virtual_ranks_reproduce_single_gpu_chain(P, world, precision):
+    wl = synth.workload("c2", L=700)
+    rows = synth.to_strings(wl["codes"])
+    N, K, seed, steps = 64, 64, wl["chain_seed"], 8
+    tree = (wl["true_parent"], wl["true_age"])
+    ref = P.Context(rows, wl["theta0"], init_tree=tree, precision=precision, max_proposals=N, max_samples=4)
+    ranks = [P.Context(rows, wl["theta0"], init_tree=tree, precision=precision, max_proposals=N, max_samples=4,
+                       rank=r, world=world) for r in range(world)]
+    for step in range(steps):
+        tr = ref.mpcgs_step_trace(step, N, K, seed)
+        for c in ranks:
+            c.mpcgs_step_local(step, N, seed)
+        full = np.concatenate([c.mpcgs_get_records(*P.mpcgs_shard_range(N, r, world)) for r, c in enumerate(ranks)])
+        assert np.array_equal(full[:, 0], tr["logL"][1:])   # bitwise: same kernels, same tiling
+        assert np.array_equal(full[:, 1], tr["S"][1:])
+        for c in ranks:
+            c.mpcgs_put_records(1, full)
+        for c in ranks:
+            assert np.array_equal(c.mpcgs_step_finish(step, N, K, seed), tr["draws"])
+        gp, ga, gl, gS = ref.mpcgs_get_state()
+        for c in ranks:
+            p2, a2, l2, S2 = c.mpcgs_get_state()
+            assert np.array_equal(p2, gp) and np.array_equal(a2, ga) and l2 == gl and S2 == gS
+
+
+def test_sample_refuses_world_gt1_without_nccl(P):
+    wl = synth.workload("c1")
+    c = P.Context(synth.to_strings(wl["codes"]), wl["theta0"], max_proposals=16, max_samples=16, rank=0, world=2)
+    with pytest.raises(P.MpcgsError) as ei:
+        c.mpcgs_sample(16, 16, 1)
+    assert ei.value.status == -3

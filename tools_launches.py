@@ -1,0 +1,12 @@
+import csv, sys
+from collections import defaultdict
+rows = list(csv.reader(open(sys.argv[1])))
+hdr = next(i for i, r in enumerate(rows) if 'Kernel Name' in r)
+h = rows[hdr]; ki = h.index('Kernel Name'); vi = h.index('Metric Value')
+d = defaultdict(list)
+for r in rows[hdr + 1:]:
+    if len(r) > vi:
+        d[r[ki][:50]].append(float(r[vi].replace(',', '')))
+tot = sum(sum(v) for v in d.values())
+for k, v in sorted(d.items(), key=lambda kv: -sum(kv[1])):
+    print(f"{k:50s} n={len(v):4d} mean={sum(v)/len(v)/1e3:9.2f} us  share={sum(v)/tot:6.3f}")
