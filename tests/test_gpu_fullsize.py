@@ -1,0 +1,69 @@
+"""Parity at BASELINE.json's full sizes, in the launch configuration bench.py
+times (one GMH step through mpcgs_step_trace with all N proposals), checked
+on outputs the oracle can compute one by one: the target, every proposal's
+resimulated times / pair code / S_G, the likelihood of a sample of proposals
+(full-alignment oracle pruning), and the draws from the GPU likelihoods
+(inverse CDF recomputed on the host from the same weights)."""
+import numpy as np
+import pytest
+
+import synth
+
+pytestmark = pytest.mark.gpu
+
+
+@pytest.fixture(scope="module")
+def P():
+    import torch
+
+    if not torch.cuda.is_available():
+        pytest.skip("no CUDA device")
+    import paper_conf_ipps_davistzw17_b200 as pkg
+
+    pkg.lib()
+    return pkg
+
+
+CASES = [
+    ("c3", {}, 3),                  # 24 x 1,000 bp, N = 256
+    ("c4", {"n": 256}, 2),          # 256 x 2,000 bp, N = 512 (largest n of the sweep)
+    ("c5", {}, 2),                  # 64 x 100,000 bp, N = 1,024 (the bench workload)
+]
+
+
+@pytest.mark.parametrize("name,over,n_ll", CASES)
+def test_full_size_step_sampled_parity(P, orc, name, over, n_ll):
+    wl = synth.workload(name, **over)
+    codes = wl["codes"]
+    n, L = codes.shape
+    N = wl["N"]
+    pi = orc.base_freqs(codes)
+    u = orc.default_rate(pi)
+    theta0 = wl["theta0"]
+    parent, age = wl["true_parent"], wl["true_age"]
+    ctx = P.Context(synth.to_strings(codes), theta0, init_tree=(parent, age), max_proposals=N, max_samples=16)
+    seed, step = wl["chain_seed"], 3
+    tr = ctx.mpcgs_step_trace(step, N, N, seed)
+    assert tr["target"] == orc.pick_target(parent, seed, step)
+    scale = age.max()
+    rng = np.random.default_rng(0)
+    ll_slots = set(rng.choice(np.arange(1, N + 1), size=n_ll, replace=False).tolist())
+    flagged = 0
+    for slot in range(1, N + 1):
+        p2, a2, t12, pair, flag = orc.propose(parent, age, theta0, tr["target"], seed, step, slot)
+        if flag:
+            flagged += 1
+            continue
+        assert tr["pair"][slot] == pair, slot
+        assert np.allclose(tr["t12"][slot], t12, rtol=0, atol=1e-12 * max(scale, t12[1]))
+        assert abs(tr["S"][slot] - orc.coalescent_S(a2, n)) <= 1e-12 * abs(tr["S"][slot])
+        if slot in ll_slots:
+            want = orc.log_likelihood(codes, p2, a2, pi, u)
+            assert abs(tr["logL"][slot] - want) <= 1e-9 * abs(want), (slot, tr["logL"][slot], want)
+    assert flagged <= 2
+    # draws: inverse CDF over softmax of the GPU likelihoods, lowest index on ties
+    w, cum = orc.weights(tr["logL"])
+    for d, got in enumerate(tr["draws"]):
+        i, near = orc.draw(cum, orc.uniform(seed, 0, step, orc.TAG_DRAW, d))
+        if not near:
+            assert got == i
