@@ -163,6 +163,7 @@ struct DevState {
     double* fixed;     // [n] sorted ages of interior nodes other than T, Par
     // proposals
     double* rec;        // [(Nmax+1)][REC]
+    int32_t* tree_need; // [Nmax] register need of each local proposal's schedule
     uint32_t* sched_op; // [Nmax][nops]
     void* sched_e;      // [Nmax][nops] x {e_a, em_a, e_b, em_b} (float or double)
     double* tile_part;  // [Nmax][tiles_max]

@@ -110,7 +110,7 @@ mpcgs_status fail(mpcgs_ctx* c, mpcgs_status st, const std::string& msg) {
 // ------------------------------------------------------------ workspace layout
 struct Layout {
     size_t codes, codes2, parent, left, right, need, age, e, em, gen, ctx_i, ctx_d, tau, len, lcnt, entry, omega, fixed;
-    size_t rec, sched_op, sched_e, tile_part, tile_cnt, sS, sL, sStep, sSlot, counters, last_draws, theta_buf,
+    size_t tree_need, rec, sched_op, sched_e, tile_part, tile_cnt, sS, sL, sStep, sSlot, counters, last_draws, theta_buf,
         theta_cnt, score_out, total;
     int tiles_max;
 };
@@ -151,6 +151,7 @@ Layout layout(int n, int L, int Nmax, int64_t Mmax, int precision) {
     y.omega = take(8 * 9 * (size_t)(n + 1));
     y.fixed = take(8 * (size_t)n);
     y.rec = take(8 * REC * (size_t)(Nmax + 1));
+    y.tree_need = take(4 * (size_t)Nmax);
     y.sched_op = take(4 * (size_t)Nmax * nops);
     y.sched_e = take(esz * (size_t)Nmax * nops);
     y.tile_part = take(8 * (size_t)Nmax * y.tiles_max);
@@ -346,7 +347,7 @@ PruneArgs prune_args(mpcgs_ctx* c, int ntrees_global, double* out, int out_first
     a.sched_op = c->s.sched_op;
     a.sched_e = c->s.sched_e;
     prune_tiling(c->L, ntrees_global, c->precision, a.tiles, a.sites_per_cta);
-    a.max_need = prune_max_need(c->n);
+    a.tree_need = c->s.tree_need;
     a.tile_part = c->s.tile_part;
     a.tile_cnt = c->s.tile_cnt;
     a.out = out;
@@ -370,6 +371,7 @@ mpcgs_status leave(mpcgs_ctx* c) {
 mpcgs_status score_batch(mpcgs_ctx* c, int count, const int32_t* parent, const double* age, double* out) {
     const int n = c->n, nn = c->nn, nops = c->nops;
     std::vector<uint32_t> ops((size_t)count * nops);
+    std::vector<int32_t> needs((size_t)count);
     std::vector<double> e8;
     std::vector<float> e4;
     if (c->precision == 32) e4.resize((size_t)count * nops * 4);
@@ -385,7 +387,9 @@ mpcgs_status score_batch(mpcgs_ctx* c, int count, const int32_t* parent, const d
                                    : host_schedule<double>(n, ht, ops.data() + (size_t)t * nops,
                                                            e8.data() + (size_t)t * nops * 4);
         if (d > c->depth) return fail(c, MPCGS_E_ARG, "tree needs more registers than compiled");
+        needs[t] = d;
     }
+    CU(cudaMemcpyAsync(c->s.tree_need, needs.data(), 4 * (size_t)count, cudaMemcpyHostToDevice, c->work));
     CU(cudaMemcpyAsync(c->s.sched_op, ops.data(), ops.size() * 4, cudaMemcpyHostToDevice, c->work));
     if (c->precision == 32)
         CU(cudaMemcpyAsync(c->s.sched_e, e4.data(), e4.size() * 4, cudaMemcpyHostToDevice, c->work));
@@ -690,6 +694,7 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
         s.omega = (double*)(b + y.omega);
         s.fixed = (double*)(b + y.fixed);
         s.rec = (double*)(b + y.rec);
+        s.tree_need = (int32_t*)(b + y.tree_need);
         s.sched_op = (uint32_t*)(b + y.sched_op);
         s.sched_e = (void*)(b + y.sched_e);
         s.tile_part = (double*)(b + y.tile_part);

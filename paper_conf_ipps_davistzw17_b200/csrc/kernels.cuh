@@ -10,6 +10,7 @@ constexpr int PRUNE_THREADS = 128;
 constexpr int PRUNE_SI64 = 2;  // sites interleaved per thread, FP64 partials
 constexpr int PRUNE_SI32 = 2;  // FP32 partials
 constexpr int PRUNE_DR = 4;    // register-resident stack levels (deeper ones spill to shared memory)
+constexpr int PRUNE_SPILL = 2; // shared-memory stack levels; trees needing more use the flat kernel
 
 struct PruneArgs {
     const uint8_t* codes;       // [n][Lpad] bytes (flat kernel)
@@ -19,7 +20,8 @@ struct PruneArgs {
     const uint32_t* sched_op;  // [ntrees][nops]
     const void* sched_e;       // [ntrees][nops] float4 / double4
     int tiles, sites_per_cta;
-    int max_need;              // largest register need of any tree in the launch (<= floor(log2 n))
+    const int32_t* tree_need;  // [ntrees] register need of each tree's schedule (nullable)
+    int need_cap;              // set by launch_prune: largest need the table kernel serves
     double* tile_part;         // [ntrees][tiles]
     uint32_t* tile_cnt;        // [ntrees], zero on entry, reset by the kernel
     double* out;               // logL of tree t -> out[(out_first + t) * out_stride]
@@ -28,6 +30,7 @@ struct PruneArgs {
 
 int prune_depth_for(int n);
 int prune_max_need(int n);
+int prune_need_cap(int n);
 int prune_batch_sites(int precision);      // sites_per_cta must be a multiple of this
 bool prune_uses_tables(int n, int precision);
 cudaError_t launch_prune(const PruneArgs& a, int ntrees, int depth, int precision, cudaStream_t st);

@@ -13,6 +13,8 @@
 // into a mantissa/exponent accumulator, so each thread takes one log at the
 // end (Eq. 22 read as a product over sites, S4).  CTA sums are reduced in a
 // fixed order by the last CTA of each tree (deterministic, P22).
+#include <algorithm>
+
 #include "common.cuh"
 #include "kernels.cuh"
 
@@ -144,6 +146,7 @@ __global__ void __launch_bounds__(PRUNE_THREADS) k_prune(PruneArgs a) {
 
     const int tree = blockIdx.y;
     const int tile = blockIdx.x;
+    if (a.tree_need && a.tree_need[tree] <= a.need_cap) return;  // scored by the table pass
     const uint32_t* __restrict__ gop = a.sched_op + (size_t)tree * a.nops;
     const E4* __restrict__ ge = reinterpret_cast<const E4*>(a.sched_e) + (size_t)tree * a.nops;
     for (int i = threadIdx.x; i < a.nops; i += blockDim.x) {
@@ -325,9 +328,8 @@ struct Stack {
 // per 32-bit word, a thread's SI sites adjacent).  The byte offset of a site's
 // table entry is one funnel rotation and one mask: rotating the word right by
 // (bit position - log2(entry bytes)) puts the 2-bit code at the entry-size bit.
-template <bool CB, int SI>
+template <int SI>
 struct Codes {
-    static_assert(!CB, "byte codes retired");
     const unsigned char* base;  // this batch's buffer
     int wofs;                   // word index of this thread's sites
     uint32_t rb[SI], ra[SI];    // rotations for the code * EB and code * 4 * EB offsets
@@ -360,27 +362,39 @@ struct Codes {
 
 constexpr uint32_t TAB_CHECK = 0x80000000u;  // toff flag: the cherry table can hold small vectors
 
-template <typename T, int DR, int SI, bool CB, int S, int DMX>
+template <typename T, int DR, int SI, bool PT, int S, int DMX>
 __device__ __forceinline__ void tab_tt(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, const T* s_tab,
-                                       const Codes<CB, SI>& c, int (&scale)[SI]) {
+                                       const Codes<SI>& c, int (&scale)[SI]) {
     if constexpr (S < DMX) {
         constexpr int EB = 4 * sizeof(T);
         const uint32_t wa = c.word((code >> 6) & 2047);
         const uint32_t wb = c.word((code >> 17) & 2047);
         const char* base = reinterpret_cast<const char*>(s_tab) + (toff & ~TAB_CHECK);
         T v[SI][4];
+        if constexpr (PT) {  // 16x4 product table of the cherry
 #pragma unroll
-        for (int k = 0; k < SI; ++k)
-            ld4<T>(v[k], reinterpret_cast<const T*>(base + c.template off4<EB>(wa, k) + c.template off<EB>(wb, k)));
-        if (toff & TAB_CHECK) rescale_sites<T, SI>(v, scale);
+            for (int k = 0; k < SI; ++k)
+                ld4<T>(v[k], reinterpret_cast<const T*>(base + c.template off4<EB>(wa, k) + c.template off<EB>(wb, k)));
+            if (toff & TAB_CHECK) rescale_sites<T, SI>(v, scale);
+        } else {             // two 4x4 tip tables, multiplied here
+#pragma unroll
+            for (int k = 0; k < SI; ++k) {
+                T w[4];
+                ld4<T>(v[k], reinterpret_cast<const T*>(base + c.template off<EB>(wa, k)));
+                ld4<T>(w, reinterpret_cast<const T*>(base + 16 * sizeof(T) + c.template off<EB>(wb, k)));
+#pragma unroll
+                for (int i = 0; i < 4; ++i) v[k][i] *= w[i];
+            }
+            rescale_sites<T, SI>(v, scale);
+        }
 #pragma unroll
         for (int k = 0; k < SI; ++k) st.template put<S>(k, v[k]);
     }
 }
 
-template <typename T, int DR, int SI, bool CB, int S, int DMX>
+template <typename T, int DR, int SI, int S, int DMX>
 __device__ __forceinline__ void tab_ts(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff,
-                                       const typename Traits<T>::E4& ed, const T* s_tab, const Codes<CB, SI>& c,
+                                       const typename Traits<T>::E4& ed, const T* s_tab, const Codes<SI>& c,
                                        const T (&pi)[4], int (&scale)[SI]) {
     if constexpr (S >= 1 && S <= DMX) {
         constexpr int EB = 4 * sizeof(T);
@@ -424,8 +438,8 @@ __device__ __forceinline__ void tab_ss(Stack<T, DR, SI>& st, const typename Trai
 }
 
 #define MPCGS_TABCASE(S)                                                                          \
-    case 3 * (S) + 0: tab_tt<T, DR, SI, CB, S, DMX>(st, code, toff, s_tab, cc, scale); break;       \
-    case 3 * (S) + 1: tab_ts<T, DR, SI, CB, S, DMX>(st, code, toff, ed, s_tab, cc, pi, scale); break; \
+    case 3 * (S) + 0: tab_tt<T, DR, SI, PT, S, DMX>(st, code, toff, s_tab, cc, scale); break;       \
+    case 3 * (S) + 1: tab_ts<T, DR, SI, S, DMX>(st, code, toff, ed, s_tab, cc, pi, scale); break;     \
     case 3 * (S) + 2: tab_ss<T, DR, SI, S, DMX>(st, ed, pi, scale); break;
 #define MPCGS_CASES_4 MPCGS_TABCASE(0) MPCGS_TABCASE(1) MPCGS_TABCASE(2) MPCGS_TABCASE(3) MPCGS_TABCASE(4)
 #define MPCGS_CASES_6 MPCGS_CASES_4 MPCGS_TABCASE(5) MPCGS_TABCASE(6)
@@ -433,9 +447,9 @@ __device__ __forceinline__ void tab_ss(Stack<T, DR, SI>& st, const typename Trai
 #define MPCGS_CASES_10 MPCGS_CASES_8 MPCGS_TABCASE(9) MPCGS_TABCASE(10)
 
 // one op for SI sites; the switch only has the (sp, type) labels a DMX-level tree can use
-template <typename T, int DR, int SI, bool CB, int DMX>
+template <typename T, int DR, int SI, bool PT, int DMX>
 __device__ __forceinline__ void run_op(int di, Stack<T, DR, SI>& st, uint32_t code, uint32_t toff,
-                                       const typename Traits<T>::E4& ed, const T* s_tab, const Codes<CB, SI>& cc,
+                                       const typename Traits<T>::E4& ed, const T* s_tab, const Codes<SI>& cc,
                                        const T (&pi)[4], int (&scale)[SI]) {
     if constexpr (DMX <= 4) {
         switch (di) { MPCGS_CASES_4 default: break; }
@@ -452,25 +466,26 @@ __host__ __device__ constexpr size_t align16(size_t x) { return (x + 15) & ~(siz
 
 // shared memory of the table kernel for trees of n tips whose register need is
 // at most `need` (spill levels above DR)
-template <typename T, int DR, int SI, bool CB>
+template <typename T, int DR, int SI, bool PT>
 __host__ __device__ size_t tab_smem_bytes(int nops, int need) {
     const int n = nops + 1;
     const int spill = need > DR ? need - DR : 0;
-    return align16(sizeof(typename Traits<T>::E4) * nops) + align16(sizeof(T) * 32 * (size_t)n) +
-           align16(sizeof(uint2) * nops) + 2 * align16(Codes<CB, SI>::buf_bytes(n)) +
+    return align16(sizeof(typename Traits<T>::E4) * nops) + align16(sizeof(T) * (PT ? 32 : 16) * (size_t)n) +
+           align16(sizeof(uint2) * nops) + 2 * align16(Codes<SI>::buf_bytes(n)) +
            sizeof(T) * (size_t)spill * SI * 4 * PRUNE_THREADS;
 }
 
-template <typename T, int DR, int SI, bool CB, int DMX>
+template <typename T, int DR, int SI, bool PT, int DMX>
 __global__ void __launch_bounds__(PRUNE_THREADS) k_prune_tab(PruneArgs a) {
     using E4 = typename Traits<T>::E4;
-    using CD = Codes<CB, SI>;
+    using CD = Codes<SI>;
+    constexpr uint32_t TABE = PT ? 32u : 16u;  // table entries per tip
     constexpr int BATCH = CD::BATCH;  // sites per batch
     extern __shared__ __align__(16) unsigned char smem_raw[];
     const int nops = a.nops, n = nops + 1;
     E4* s_e = reinterpret_cast<E4*>(smem_raw);
     T* s_tab = reinterpret_cast<T*>(smem_raw + align16(sizeof(E4) * nops));
-    uint2* s_op = reinterpret_cast<uint2*>(reinterpret_cast<unsigned char*>(s_tab) + align16(sizeof(T) * 32 * n));
+    uint2* s_op = reinterpret_cast<uint2*>(reinterpret_cast<unsigned char*>(s_tab) + align16(sizeof(T) * TABE * n));
     unsigned char* s_cod = reinterpret_cast<unsigned char*>(s_op) + align16(sizeof(uint2) * nops);
     const size_t bufb = align16(CD::buf_bytes(n));
     T* s_spill = reinterpret_cast<T*>(s_cod + 2 * bufb);
@@ -483,6 +498,7 @@ __global__ void __launch_bounds__(PRUNE_THREADS) k_prune_tab(PruneArgs a) {
     const int s_begin = tile * a.sites_per_cta;
     const int s_end = min(a.L, s_begin + a.sites_per_cta);
     const int nb = (s_end - s_begin + BATCH - 1) / BATCH;
+    if (a.tree_need && a.tree_need[tree] > a.need_cap) return;  // deeper tree: scored by the flat pass
 
     auto issue = [&](int b, int buf) {
         const int site0 = s_begin + b * BATCH;
@@ -512,7 +528,7 @@ __global__ void __launch_bounds__(PRUNE_THREADS) k_prune_tab(PruneArgs a) {
             uint32_t sz = 0;
             if (i < nops) {
                 const uint32_t ty = s_op[i].x & 3u;
-                sz = ty == OP_TT ? 64u : (ty == OP_TS ? 16u : 0u);
+                sz = ty == OP_TT ? 2u * TABE : (ty == OP_TS ? 16u : 0u);
             }
             uint32_t x = sz;
 #pragma unroll
@@ -531,12 +547,16 @@ __global__ void __launch_bounds__(PRUNE_THREADS) k_prune_tab(PruneArgs a) {
         const uint32_t ty = s_op[op].x & 3u;
         T* tab = reinterpret_cast<T*>(reinterpret_cast<char*>(s_tab) + s_op[op].y);
         const E4 ed = s_e[op];
-        if (ty == OP_TT) {
+        if (ty == OP_TT && PT) {
             // cherry: entry (xa, xb) = P_{.,xa}(t_a) (.) P_{.,xb}(t_b)   (Eq. 19-20 at two tips)
             const int xa = j >> 4, xb = (j >> 2) & 3, X = j & 3;
             const T va = (X == xa ? (T)ed.x : T(0)) + (T)ed.y * pick4(pi, xa);
             const T vb = (X == xb ? (T)ed.z : T(0)) + (T)ed.w * pick4(pi, xb);
             tab[j] = va * vb;
+        } else if (ty == OP_TT && j < 32) {  // two tip tables: a at [0, 16), b at [16, 32)
+            const int x = (j >> 2) & 3, X = j & 3;
+            tab[j] = j < 16 ? (X == x ? (T)ed.x : T(0)) + (T)ed.y * pick4(pi, x)
+                            : (X == x ? (T)ed.z : T(0)) + (T)ed.w * pick4(pi, x);
         } else if (ty == OP_TS && j < 16) {
             const int x = j >> 2, X = j & 3;
             tab[j] = (X == x ? (T)ed.x : T(0)) + (T)ed.y * pick4(pi, x);
@@ -544,7 +564,7 @@ __global__ void __launch_bounds__(PRUNE_THREADS) k_prune_tab(PruneArgs a) {
     }
     __syncthreads();
     // flag cherry tables with an entry whose max is below the rescale threshold
-    for (int op = tid; op < nops; op += PRUNE_THREADS) {
+    for (int op = tid; op < nops && PT; op += PRUNE_THREADS) {
         if ((s_op[op].x & 3u) != OP_TT) continue;
         const T* tab = reinterpret_cast<const T*>(reinterpret_cast<const char*>(s_tab) + s_op[op].y);
         bool small = false;
@@ -585,7 +605,7 @@ __global__ void __launch_bounds__(PRUNE_THREADS) k_prune_tab(PruneArgs a) {
             const uint2 ox = s_op[op];
             const E4 ed = s_e[op];
             const int di = (int)((ox.x >> 2) & 15u) * 3 + (int)(ox.x & 3u);  // dense (sp, type) index
-            run_op<T, DR, SI, CB, DMX>(di, st, ox.x, ox.y, ed, s_tab, cc, pi, scale);
+            run_op<T, DR, SI, PT, DMX>(di, st, ox.x, ox.y, ed, s_tab, cc, pi, scale);
         }
         const int site0 = s_begin + b * BATCH + tid * SI;
 #pragma unroll
@@ -649,10 +669,10 @@ static cudaError_t launch_flat(const PruneArgs& a, int ntrees, cudaStream_t st) 
     return cudaGetLastError();
 }
 
-template <typename T, int DR, int SI, bool CB, int DMX>
+template <typename T, int DR, int SI, bool PT, int DMX>
 static cudaError_t launch_tab(const PruneArgs& a, int ntrees, cudaStream_t st) {
-    const size_t smem = tab_smem_bytes<T, DR, SI, CB>(a.nops, a.max_need);
-    auto kern = k_prune_tab<T, DR, SI, CB, DMX>;
+    const size_t smem = tab_smem_bytes<T, DR, SI, PT>(a.nops, a.need_cap);
+    auto kern = k_prune_tab<T, DR, SI, PT, DMX>;
     static size_t attr_bytes = 48 * 1024;
     if (smem > attr_bytes) {
         cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
@@ -681,28 +701,37 @@ int prune_max_need(int n) {
 
 int prune_batch_sites(int precision) { return PRUNE_THREADS * (precision == 32 ? PRUNE_SI32 : PRUNE_SI64); }
 
-bool prune_code_bytes(int, int) { return false; }
+// register need the table kernel serves (DR registers + PRUNE_SPILL shared levels);
+// deeper trees (rare) are scored by the flat kernel in a second pass
+int prune_need_cap(int n) { return std::min(prune_max_need(n), PRUNE_DR + PRUNE_SPILL); }
+
+static bool product_tables(int n) { return n <= 128; }
 
 bool prune_uses_tables(int n, int precision) {
-    const int need = prune_max_need(n);
-    const size_t bytes = precision == 32 ? tab_smem_bytes<float, PRUNE_DR, PRUNE_SI32, false>(n - 1, need)
-                                         : tab_smem_bytes<double, PRUNE_DR, PRUNE_SI64, false>(n - 1, need);
+    const int cap = prune_need_cap(n);
+    const bool pt = product_tables(n);
+    size_t bytes;
+    if (precision == 32)
+        bytes = pt ? tab_smem_bytes<float, PRUNE_DR, PRUNE_SI32, true>(n - 1, cap)
+                   : tab_smem_bytes<float, PRUNE_DR, PRUNE_SI32, false>(n - 1, cap);
+    else
+        bytes = pt ? tab_smem_bytes<double, PRUNE_DR, PRUNE_SI64, true>(n - 1, cap)
+                   : tab_smem_bytes<double, PRUNE_DR, PRUNE_SI64, false>(n - 1, cap);
     return bytes <= 160 * 1024;
 }
 
-template <typename T, int SI, bool CB>
-static cudaError_t launch_tab_dmx(const PruneArgs& a, int ntrees, int depth, cudaStream_t st) {
-    switch (depth) {
-        case 4: return launch_tab<T, PRUNE_DR, SI, CB, 4>(a, ntrees, st);
-        case 6: return launch_tab<T, PRUNE_DR, SI, CB, 6>(a, ntrees, st);
-        case 8: return launch_tab<T, PRUNE_DR, SI, CB, 8>(a, ntrees, st);
-        default: return launch_tab<T, PRUNE_DR, SI, CB, 10>(a, ntrees, st);
+template <typename T, int SI, bool PT>
+static cudaError_t launch_tab_dmx(const PruneArgs& a, int ntrees, cudaStream_t st) {
+    switch (a.need_cap) {
+        case 1: case 2: case 3: case 4: return launch_tab<T, PRUNE_DR, SI, PT, 4>(a, ntrees, st);
+        case 5: case 6: return launch_tab<T, PRUNE_DR, SI, PT, 6>(a, ntrees, st);
+        case 7: case 8: return launch_tab<T, PRUNE_DR, SI, PT, 8>(a, ntrees, st);
+        default: return launch_tab<T, PRUNE_DR, SI, PT, 10>(a, ntrees, st);
     }
 }
 
-template <typename T, int SI>
-static cudaError_t launch_typed(const PruneArgs& a, int ntrees, int depth, bool tab, cudaStream_t st) {
-    if (tab) return launch_tab_dmx<T, SI, false>(a, ntrees, depth, st);
+template <typename T>
+static cudaError_t launch_flat_depth(const PruneArgs& a, int ntrees, int depth, cudaStream_t st) {
     switch (depth) {
         case 4: return launch_flat<T, 4>(a, ntrees, st);
         case 6: return launch_flat<T, 6>(a, ntrees, st);
@@ -711,11 +740,26 @@ static cudaError_t launch_typed(const PruneArgs& a, int ntrees, int depth, bool 
     }
 }
 
+template <typename T, int SI>
+static cudaError_t launch_typed(PruneArgs a, int ntrees, int depth, cudaStream_t st) {
+    const int n = a.nops + 1;
+    if (a.codes2 == nullptr || !prune_uses_tables(n, sizeof(T) == 4 ? 32 : 64)) {
+        a.tree_need = nullptr;  // flat kernel for every tree
+        return launch_flat_depth<T>(a, ntrees, depth, st);
+    }
+    a.need_cap = prune_need_cap(n);
+    const bool deep = prune_max_need(n) > a.need_cap && a.tree_need != nullptr;
+    if (!deep) a.tree_need = nullptr;
+    cudaError_t e = product_tables(n) ? launch_tab_dmx<T, SI, true>(a, ntrees, st)
+                                      : launch_tab_dmx<T, SI, false>(a, ntrees, st);
+    if (e != cudaSuccess || !deep) return e;
+    return launch_flat_depth<T>(a, ntrees, depth, st);  // trees with need > cap only
+}
+
 cudaError_t launch_prune(const PruneArgs& a, int ntrees, int depth, int precision, cudaStream_t st) {
     if (ntrees <= 0) return cudaSuccess;
-    const bool tab = a.codes2 != nullptr && prune_uses_tables(a.nops + 1, precision);
-    if (precision == 32) return launch_typed<float, PRUNE_SI32>(a, ntrees, depth, tab, st);
-    return launch_typed<double, PRUNE_SI64>(a, ntrees, depth, tab, st);
+    if (precision == 32) return launch_typed<float, PRUNE_SI32>(a, ntrees, depth, st);
+    return launch_typed<double, PRUNE_SI64>(a, ntrees, depth, st);
 }
 
 }  // namespace mpcgs

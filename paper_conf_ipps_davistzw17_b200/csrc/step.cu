@@ -480,6 +480,7 @@ __global__ void __launch_bounds__(32) k_propose(DevState s, uint64_t seed, int64
         sNeed[T] = su_need(sNeed[x], sNeed[y]);
         sNeed[Par] = su_need(sNeed[T], sNeed[z]);
         for (int v = A; v >= 0; v = s.parent[v]) sNeed[v] = su_need(sNeed[sL[v - n]], sNeed[sR[v - n]]);
+        s.tree_need[local] = sNeed[root];
     } else if (lane == 1) {
         sh_d[2] = exp(-u * (t1 - s.age[x]));
         sh_d[3] = -expm1(-u * (t1 - s.age[x]));
