@@ -435,15 +435,16 @@ mpcgs_status check_status(mpcgs_ctx* c) {
 
 // one step's proposal work for this rank: context, propose, prune
 mpcgs_status step_local_launch(mpcgs_ctx* c, uint64_t seed, int64_t step, int N, cudaEvent_t pre = nullptr,
-                               cudaEvent_t post = nullptr) {
+                               cudaEvent_t post = nullptr, bool with_context = true) {
     int first = 1 + c->rank * (N / c->world), count = N / c->world;
-    CU(launch_context(c->s, seed, step, c->work));
+    if (with_context) CU(launch_context(c->s, seed, step, c->work));
     CU(launch_propose(c->s, seed, step, first, count, c->work));
     PruneArgs a = prune_args(c, N, c->s.rec, first, REC);
     if (pre) CU(cudaEventRecord(pre, c->work));
-    CU(launch_prune(a, count, c->depth, c->precision, c->work));
+    int np = 0;
+    CU(launch_prune(a, count, c->depth, c->precision, c->work, &np));
     if (post) CU(cudaEventRecord(post, c->work));
-    c->launches += 3;
+    c->launches += (with_context ? 2 : 1) + np;
     return MPCGS_OK;
 }
 
@@ -782,10 +783,10 @@ mpcgs_status mpcgs_sample(mpcgs_ctx* c, int32_t N, int64_t M, uint64_t seed) {
     c->launches = 0;
     c->prune_ms = 0.0;
     auto one_step = [&]() -> mpcgs_status {
-        mpcgs_status s2 = step_local_launch(c, seed, -1, N);
+        mpcgs_status s2 = step_local_launch(c, seed, -1, N, nullptr, nullptr, false);
         if (s2) return s2;
         if ((s2 = allgather_records(c, N))) return s2;
-        CU(launch_draw(c->s, seed, -1, N, -1, c->burnin, M, c->work));
+        CU(launch_draw(c->s, seed, -1, N, -1, c->burnin, M, steps, c->work));
         ++c->launches;
         return MPCGS_OK;
     };
@@ -802,9 +803,13 @@ mpcgs_status mpcgs_sample(mpcgs_ctx* c, int32_t N, int64_t M, uint64_t seed) {
             if ((c->timing & 2) && c->flush_buf)
                 CU(cudaMemsetAsync(c->flush_buf, (int)(k & 0xff), (size_t)256 << 20, c->work));
             CU(cudaEventRecord(c->evpool[4 * k + 0], c->work));
-            if ((st = step_local_launch(c, seed, -1, N, c->evpool[4 * k + 1], c->evpool[4 * k + 2]))) return st;
+            if (k == 0) {  // the first context; later ones come from k_draw
+                CU(launch_context(c->s, seed, -1, c->work));
+                ++c->launches;
+            }
+            if ((st = step_local_launch(c, seed, -1, N, c->evpool[4 * k + 1], c->evpool[4 * k + 2], false))) return st;
             if ((st = allgather_records(c, N))) return st;
-            CU(launch_draw(c->s, seed, -1, N, -1, c->burnin, M, c->work));
+            CU(launch_draw(c->s, seed, -1, N, -1, c->burnin, M, steps, c->work));
             ++c->launches;
             CU(cudaEventRecord(c->evpool[4 * k + 3], c->work));
         }
@@ -826,7 +831,12 @@ mpcgs_status mpcgs_sample(mpcgs_ctx* c, int32_t N, int64_t M, uint64_t seed) {
         cudaGraph_t graph = nullptr;
         cudaGraphExec_t exec = nullptr;
         const int64_t reps = steps / G, rest = steps % G;
+        CU(cudaEventRecord(c->ev_b, c->work));
+        CU(launch_context(c->s, seed, -1, c->work));  // the first context; later ones come from k_draw
+        c->launches = 1;
+        int64_t per_graph = 0;
         if (reps > 0) {
+            const int64_t before = c->launches;
             CU(cudaStreamBeginCapture(c->work, cudaStreamCaptureModeThreadLocal));
             for (int64_t k = 0; k < G; ++k) {
                 if ((st = one_step())) {
@@ -837,12 +847,12 @@ mpcgs_status mpcgs_sample(mpcgs_ctx* c, int32_t N, int64_t M, uint64_t seed) {
             }
             CU(cudaStreamEndCapture(c->work, &graph));
             CU(cudaGraphInstantiate(&exec, graph, 0));
-            c->launches = 0;
+            per_graph = c->launches - before;
+            c->launches = before;
         }
-        CU(cudaEventRecord(c->ev_b, c->work));
         for (int64_t r = 0; r < reps; ++r) {
             CU(cudaGraphLaunch(exec, c->work));
-            c->launches += 4 * G;
+            c->launches += per_graph;
         }
         for (int64_t k = 0; k < rest; ++k)
             if ((st = one_step())) return st;
@@ -952,7 +962,7 @@ mpcgs_status mpcgs_step_finish(mpcgs_ctx* c, int64_t step, int32_t N, int32_t K,
     mpcgs_status st = enter(c);
     if (st) return st;
     CU(cudaMemsetAsync(c->s.counters + 2, 0, 8, c->work));
-    CU(launch_draw(c->s, seed, step, N, K, 0, 0, c->work));
+    CU(launch_draw(c->s, seed, step, N, K, 0, 0, 0, c->work));
     if (draws) CU(cudaMemcpyAsync(draws, c->s.last_draws, 4 * (size_t)K, cudaMemcpyDeviceToHost, c->work));
     if ((st = leave(c))) return st;
     return check_status(c);
@@ -967,7 +977,7 @@ mpcgs_status mpcgs_step_trace(mpcgs_ctx* c, int64_t step, int32_t N, int32_t K, 
     if (st) return st;
     CU(cudaMemsetAsync(c->s.counters + 2, 0, 8, c->work));
     if ((st = step_local_launch(c, seed, step, N))) return st;
-    CU(launch_draw(c->s, seed, step, N, K, 0, 0, c->work));
+    CU(launch_draw(c->s, seed, step, N, K, 0, 0, 0, c->work));
     std::vector<double> rec((size_t)(N + 1) * REC);
     int32_t ci[16];
     CU(cudaMemcpyAsync(rec.data(), c->s.rec, rec.size() * 8, cudaMemcpyDeviceToHost, c->work));

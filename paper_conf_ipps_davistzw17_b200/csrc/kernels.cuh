@@ -33,15 +33,17 @@ int prune_max_need(int n);
 int prune_need_cap(int n);
 int prune_batch_sites(int precision);      // sites_per_cta must be a multiple of this
 bool prune_uses_tables(int n, int precision);
-cudaError_t launch_prune(const PruneArgs& a, int ntrees, int depth, int precision, cudaStream_t st);
+cudaError_t launch_prune(const PruneArgs& a, int ntrees, int depth, int precision, cudaStream_t st,
+                         int* n_launched = nullptr);
 
 // step kernels (step.cu); step < 0 -> read the step index from counters[0]
 cudaError_t launch_context(const DevState& s, uint64_t seed, int64_t step, cudaStream_t st);
 cudaError_t launch_propose(const DevState& s, uint64_t seed, int64_t step, int slot_first, int count,
                            cudaStream_t st);
 // draw: K < 0 -> loop mode (burn-in / sampling from counters, store, advance step)
+// loop mode also computes the context of step+1 when step+1 < total_steps
 cudaError_t launch_draw(const DevState& s, uint64_t seed, int64_t step, int N, int K, int burnin,
-                        int64_t M, cudaStream_t st);
+                        int64_t M, int64_t total_steps, cudaStream_t st);
 cudaError_t launch_fill_gen_record(const DevState& s, cudaStream_t st);
 
 // theta kernels (theta.cu)

@@ -741,8 +741,9 @@ static cudaError_t launch_flat_depth(const PruneArgs& a, int ntrees, int depth, 
 }
 
 template <typename T, int SI>
-static cudaError_t launch_typed(PruneArgs a, int ntrees, int depth, cudaStream_t st) {
+static cudaError_t launch_typed(PruneArgs a, int ntrees, int depth, cudaStream_t st, int& nl) {
     const int n = a.nops + 1;
+    nl = 1;
     if (a.codes2 == nullptr || !prune_uses_tables(n, sizeof(T) == 4 ? 32 : 64)) {
         a.tree_need = nullptr;  // flat kernel for every tree
         return launch_flat_depth<T>(a, ntrees, depth, st);
@@ -753,13 +754,19 @@ static cudaError_t launch_typed(PruneArgs a, int ntrees, int depth, cudaStream_t
     cudaError_t e = product_tables(n) ? launch_tab_dmx<T, SI, true>(a, ntrees, st)
                                       : launch_tab_dmx<T, SI, false>(a, ntrees, st);
     if (e != cudaSuccess || !deep) return e;
+    nl = 2;
     return launch_flat_depth<T>(a, ntrees, depth, st);  // trees with need > cap only
 }
 
-cudaError_t launch_prune(const PruneArgs& a, int ntrees, int depth, int precision, cudaStream_t st) {
-    if (ntrees <= 0) return cudaSuccess;
-    if (precision == 32) return launch_typed<float, PRUNE_SI32>(a, ntrees, depth, st);
-    return launch_typed<double, PRUNE_SI64>(a, ntrees, depth, st);
+cudaError_t launch_prune(const PruneArgs& a, int ntrees, int depth, int precision, cudaStream_t st,
+                         int* n_launched) {
+    int nl = 0;
+    cudaError_t e = cudaSuccess;
+    if (ntrees > 0)
+        e = precision == 32 ? launch_typed<float, PRUNE_SI32>(a, ntrees, depth, st, nl)
+                            : launch_typed<double, PRUNE_SI64>(a, ntrees, depth, st, nl);
+    if (n_launched) *n_launched = nl;
+    return e;
 }
 
 }  // namespace mpcgs

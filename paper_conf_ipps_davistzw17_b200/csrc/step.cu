@@ -11,6 +11,7 @@
 //   k_draw     (1 CTA)      weights = softmax(logL) over N+1 states (Eq. 29-31,
 //                           S18: the prior is recorded, never added), K inverse-
 //                           CDF draws (L1140-1144), sample store, generator commit
+#include <algorithm>
 #include <cfloat>
 
 #include "common.cuh"
@@ -96,8 +97,11 @@ __device__ int block_exclusive_scan(int v, int* s_warp, int* tot) {
 }
 
 // ------------------------------------------------------------------ k_context
-__global__ void __launch_bounds__(CTX_THREADS) k_context(DevState s, uint64_t seed, int64_t step_arg) {
-    extern __shared__ __align__(16) double csm[];
+// Block-wide context computation, NT threads; csm = dynamic shared memory of
+// context_smem_bytes(n).  Used by k_context and, for the next step of the
+// device loop, at the end of k_draw (saves a launch per step).
+template <int NT>
+__device__ void context_body(const DevState& s, uint64_t seed, int64_t step_arg, double* csm) {
     const int n = s.n, nn = s.nn, nint = n - 1;
     double* sAge = csm;               // [n-1] ages of interior nodes (index v - n)
     double* sF = sAge + nint;         // [n] sorted fixed ages
@@ -108,10 +112,10 @@ __global__ void __launch_bounds__(CTX_THREADS) k_context(DevState s, uint64_t se
     int* sEntry = reinterpret_cast<int*>(sBeta + 3 * (n + 1));  // [n+1]
     __shared__ int sh[16];
     __shared__ double shd[8];
-    __shared__ int s_warp[CTX_THREADS / 32];
+    __shared__ int s_warp[NT / 32];
     const int tid = threadIdx.x;
 
-    for (int i = tid; i < nint; i += CTX_THREADS) {
+    for (int i = tid; i < nint; i += NT) {
         sAge[i] = s.age[n + i];
         if (s.parent[n + i] < 0) sh[10] = n + i;  // root
     }
@@ -147,7 +151,7 @@ __global__ void __launch_bounds__(CTX_THREADS) k_context(DevState s, uint64_t se
     const int nfixed = n - 3;
 
     // rank sort of the fixed interior nodes by (age, id)
-    for (int v = n + tid; v < nn; v += CTX_THREADS) {
+    for (int v = n + tid; v < nn; v += NT) {
         if (v == T || v == Par) continue;
         const double av = sAge[v - n];
         int r = 0;
@@ -170,7 +174,7 @@ __global__ void __launch_bounds__(CTX_THREADS) k_context(DevState s, uint64_t se
     }
     __syncthreads();
     const int lo = sh[11], cnt = sh[12], ins = sh[13], has3 = sh[14];
-    for (int j = tid; j < cnt; j += CTX_THREADS) {
+    for (int j = tid; j < cnt; j += NT) {
         double x;
         if (!has3) x = sF[lo + j];
         else if (j < ins) x = sF[lo + j];
@@ -181,11 +185,11 @@ __global__ void __launch_bounds__(CTX_THREADS) k_context(DevState s, uint64_t se
     __syncthreads();
     // dedupe (equal ages are one cut) by an exclusive scan of keep flags
     int carry = 0;
-    for (int base = 0; base < cnt; base += CTX_THREADS) {
+    for (int base = 0; base < cnt; base += NT) {
         const int j = base + tid;
         const int keep = (j < cnt) && (j == 0 || sX[j] != sX[j - 1]);
         int tot;
-        const int pos = block_exclusive_scan<CTX_THREADS>(keep, s_warp, &tot);
+        const int pos = block_exclusive_scan<NT>(keep, s_warp, &tot);
         if (keep) sTau[1 + carry + pos] = sX[j];
         carry += tot;
     }
@@ -196,7 +200,7 @@ __global__ void __launch_bounds__(CTX_THREADS) k_context(DevState s, uint64_t se
     }
     __syncthreads();
     // per-interval bookkeeping and closed-form weights
-    for (int p = tid; p < m; p += CTX_THREADS) {
+    for (int p = tid; p < m; p += NT) {
         const double tp = sTau[p];
         const bool inf = rootcase && p == m - 1;
         const double len = inf ? CUDART_INF : sTau[p + 1] - tp;
@@ -240,7 +244,7 @@ __global__ void __launch_bounds__(CTX_THREADS) k_context(DevState s, uint64_t se
     }
     __syncthreads();
     // forward choice weights omega_p(k -> k') = W^_p(k -> k') beta_{p+1}(k' + entry_{p+1})
-    for (int p = tid; p < m; p += CTX_THREADS) {
+    for (int p = tid; p < m; p += NT) {
         const int en = sEntry[p + 1];
         const double* bn = sBeta + (p + 1) * 3;
         const double be1 = en ? bn[1] : bn[0], be2 = en ? bn[2] : bn[1], be3 = en ? 0.0 : bn[2];
@@ -251,7 +255,7 @@ __global__ void __launch_bounds__(CTX_THREADS) k_context(DevState s, uint64_t se
         om[6] = W[5] * be1; om[7] = W[4] * be2;  om[8] = W[3] * be3;
         s.entry[p] = sEntry[p];
     }
-    for (int i = tid; i < nfixed; i += CTX_THREADS) s.fixed[i] = sF[i];
+    for (int i = tid; i < nfixed; i += NT) s.fixed[i] = sF[i];
     if (tid == 0) {
         s.tau[m] = tA;
         s.entry[m] = 0;
@@ -262,6 +266,11 @@ __global__ void __launch_bounds__(CTX_THREADS) k_context(DevState s, uint64_t se
         for (int i = 0; i < 4; ++i) s.ctx_d[i] = shd[i];
         s.counters[4] = T;
     }
+}
+
+__global__ void __launch_bounds__(CTX_THREADS) k_context(DevState s, uint64_t seed, int64_t step_arg) {
+    extern __shared__ __align__(16) double csm[];
+    context_body<CTX_THREADS>(s, seed, step_arg, csm);
 }
 
 size_t context_smem_bytes(int n) {
@@ -342,9 +351,26 @@ struct WalkCtx {  // the step's interval context, staged in shared memory
     double theta0;
 };
 
+// uniforms of the slot's stream: the first PRE_U precomputed by the warp's lanes
+constexpr int PRE_U = 64;
+struct PreStream {
+    const double* pre;
+    UStream us;
+    __device__ PreStream(const double* p, uint64_t seed, uint32_t slot, uint32_t step)
+        : pre(p), us(seed, slot, step, TAG_PROPOSE) {}
+    __device__ __forceinline__ double next() {
+        const uint32_t i = us.idx;
+        if (i < (uint32_t)PRE_U) {
+            ++us.idx;
+            return pre[i];
+        }
+        return us.next();
+    }
+};
+
 __device__ Walk forward_walk(const WalkCtx& s, int m, int k0, bool rootcase, uint64_t seed, uint32_t slot,
-                             uint32_t step) {
-    UStream us(seed, slot, step, TAG_PROPOSE);
+                             uint32_t step, const double* pre_u) {
+    PreStream us(pre_u, seed, slot, step);
     Walk w{0.0, 0.0, 0, 0};
     double tt[2] = {0.0, 0.0};
     int k = k0, events = 0;
@@ -419,6 +445,7 @@ __global__ void __launch_bounds__(32) k_propose(DevState s, uint64_t seed, int64
     double* sOm = sLen + n + 1;    // [9(n+1)]
     __shared__ double sh_d[8];  // t1, t2, e/em of changed branches
     __shared__ int sh_i[8];
+    __shared__ double sU[PRE_U];  // first uniforms of this slot's Philox stream
     const int lane = threadIdx.x;
     const int slot = slot_first + blockIdx.x;  // global slot 1..N
     const int local = blockIdx.x;
@@ -440,10 +467,16 @@ __global__ void __launch_bounds__(32) k_propose(DevState s, uint64_t seed, int64
         }
     }
     for (int i = lane; i < 9 * m; i += 32) sOm[i] = s.omega[i];
+    {  // one Philox block per lane: uniforms 2*lane, 2*lane+1 of (slot, step, PROPOSE)
+        const U4 b = philox(U4{(uint32_t)lane, (uint32_t)slot, (uint32_t)step, TAG_PROPOSE}, (uint32_t)seed,
+                            (uint32_t)(seed >> 32));
+        sU[2 * lane] = to_unit(b.x, b.y);
+        sU[2 * lane + 1] = to_unit(b.z, b.w);
+    }
     __syncwarp();
     if (lane == 0) {
         const WalkCtx wc{sTau, sLen, sOm, sLc, sEn, s.theta0};
-        Walk w = forward_walk(wc, m, k0, rootcase, seed, (uint32_t)slot, (uint32_t)step);
+        Walk w = forward_walk(wc, m, k0, rootcase, seed, (uint32_t)slot, (uint32_t)step, sU);
         int pair = w.pair;
         double t1 = w.t1, t2 = w.t2;
         if (!w.ok) {
@@ -585,7 +618,7 @@ cudaError_t launch_propose(const DevState& s, uint64_t seed, int64_t step, int s
 
 // ------------------------------------------------------------------ k_draw
 __global__ void __launch_bounds__(DRAW_THREADS) k_draw(DevState s, uint64_t seed, int64_t step_arg, int N,
-                                                       int K_arg, int burnin, int64_t M) {
+                                                       int K_arg, int burnin, int64_t M, int64_t total_steps) {
     extern __shared__ __align__(16) double dsm[];
     double* sC = dsm;  // [N+1] cumulative weights
     __shared__ double s_red[DRAW_THREADS / 32];
@@ -693,10 +726,9 @@ __global__ void __launch_bounds__(DRAW_THREADS) k_draw(DevState s, uint64_t seed
         }
     }
     __syncthreads();
-    if (tid != 0) return;
     // commit: the last draw generates the next proposal set (Fig. 12)
     const int I = K > 0 ? s.last_draws[K - 1] : 0;
-    if (I > 0) {
+    if (tid == 0 && I > 0) {
         const double* r = s.rec + (size_t)I * REC;
         const int A = s.ctx_i[2];
         const int c0 = s.ctx_i[6], c1 = s.ctx_i[7], c2 = s.ctx_i[8];
@@ -734,17 +766,30 @@ __global__ void __launch_bounds__(DRAW_THREADS) k_draw(DevState s, uint64_t seed
         s.gen[0] = r[0];
         s.gen[1] = r[1];
     }
-    if (K_arg < 0) {
-        s.counters[0] = step + 1;
-        if (s_store) s.counters[1] = stored + K;
+    if (tid == 0) {
+        if (K_arg < 0) {
+            s.counters[0] = step + 1;
+            if (s_store) s.counters[1] = stored + K;
+        }
+        s.counters[3] = K;
     }
-    s.counters[3] = K;
+    // device loop: the next step's context, from the committed generator
+    if (K_arg < 0 && step + 1 < total_steps) {
+        __syncthreads();
+        context_body<DRAW_THREADS>(s, seed, step + 1, dsm);
+    }
 }
 
 cudaError_t launch_draw(const DevState& s, uint64_t seed, int64_t step, int N, int K, int burnin, int64_t M,
-                        cudaStream_t st) {
-    size_t smem = sizeof(double) * (size_t)(N + 1);
-    k_draw<<<1, DRAW_THREADS, smem, st>>>(s, seed, step, N, K, burnin, M);
+                        int64_t total_steps, cudaStream_t st) {
+    const size_t smem = std::max(sizeof(double) * (size_t)(N + 1), context_smem_bytes(s.n));
+    static size_t attr_bytes = 48 * 1024;
+    if (smem > attr_bytes) {
+        cudaError_t e = cudaFuncSetAttribute(k_draw, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+        if (e != cudaSuccess) return e;
+        attr_bytes = smem;
+    }
+    k_draw<<<1, DRAW_THREADS, smem, st>>>(s, seed, step, N, K, burnin, M, total_steps);
     return cudaGetLastError();
 }
 
