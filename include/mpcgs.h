@@ -167,6 +167,13 @@ int64_t mpcgs_num_samples(const mpcgs_ctx* ctx);
 /* Re-drive: theta0 <- theta (L791-797).  Cached P(D|G) stays valid (Eq. 23). */
 mpcgs_status mpcgs_set_theta0(mpcgs_ctx* ctx, double theta0);
 
+/* EM loop of Fig. 11 (L1208-1225, L791-797): n_iter times { burn-in + sample
+ * (n_proposals, n_samples, seed + it); theta-hat over a n_grid grid;
+ * theta0 <- theta-hat }.  theta_trace: host [n_iter] (nullable) receives each
+ * iteration's estimate; the chain state carries over between iterations. */
+mpcgs_status mpcgs_em(mpcgs_ctx* ctx, int32_t n_iter, int32_t n_proposals, int64_t n_samples,
+                      uint64_t seed, int32_t n_grid, double* theta_trace);
+
 /* Model parameters actually used (host out: pi[4], u). */
 mpcgs_status mpcgs_get_model(const mpcgs_ctx* ctx, double* pi, double* mu);
 

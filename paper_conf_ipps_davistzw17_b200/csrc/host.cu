@@ -1004,6 +1004,21 @@ mpcgs_status mpcgs_set_theta0(mpcgs_ctx* c, double theta0) {
     return MPCGS_OK;
 }
 
+mpcgs_status mpcgs_em(mpcgs_ctx* c, int32_t n_iter, int32_t N, int64_t M, uint64_t seed, int32_t G,
+                      double* theta_trace) {
+    CHECK_CTX(c);
+    if (n_iter < 1 || M < 1) return fail(c, MPCGS_E_ARG, "em: n_iter and n_samples must be positive");
+    for (int32_t it = 0; it < n_iter; ++it) {
+        mpcgs_status st = mpcgs_sample(c, N, M, seed + (uint64_t)it);
+        if (st) return st;
+        double th = 0.0;
+        if ((st = mpcgs_estimate_theta(c, &th, G, nullptr, nullptr))) return st;
+        if (theta_trace) theta_trace[it] = th;
+        if ((st = mpcgs_set_theta0(c, th))) return st;
+    }
+    return MPCGS_OK;
+}
+
 mpcgs_status mpcgs_get_model(const mpcgs_ctx* c, double* pi, double* mu) {
     if (!c) return MPCGS_E_ARG;
     if (pi)

@@ -66,6 +66,7 @@ _SIGS = {
     "mpcgs_get_samples": (_i32, [_P, _i64, _i64, _P, _P, _P, _P]),
     "mpcgs_num_samples": (_i64, [_P]),
     "mpcgs_set_theta0": (_i32, [_P, _f64]),
+    "mpcgs_em": (_i32, [_P, _i32, _i32, _i64, _u64, _i32, _P]),
     "mpcgs_get_model": (_i32, [_P, _P, _P]),
     "mpcgs_set_timing": (_i32, [_P, _i32]),
     "mpcgs_last_timing": (_i32, [_P, _P, _P, _P]),
@@ -333,6 +334,11 @@ class Context:
 
     def mpcgs_set_theta0(self, theta0):
         self._chk(lib().mpcgs_set_theta0(self.h, theta0), "set_theta0")
+
+    def mpcgs_em(self, n_iter, n_proposals, n_samples, seed, n_grid=256):
+        trace = np.zeros(n_iter)
+        self._chk(lib().mpcgs_em(self.h, n_iter, n_proposals, n_samples, seed, n_grid, _ptr(trace)), "em")
+        return trace
 
     def mpcgs_get_model(self):
         pi = np.zeros(4)

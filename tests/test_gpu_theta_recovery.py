@@ -1,0 +1,49 @@
+"""theta recovery (the shape of Table 1, without
+LAMARC): data simulated under the coalescent + F81 (synth/), the EM loop of
+Fig. 11 (L1208-1225) driven from theta0 = 0.01 (Fig. 5's driving value,
+L786-788).  With 10 kbp alignments the posterior concentrates on the true
+genealogy, so theta-hat must approach the single-tree MLE S(G_true)/(n-1);
+across replicates theta-hat tracks theta_true (Pearson r, cf. r = 0.905 at
+L1533-1535)."""
+import numpy as np
+import pytest
+
+import synth
+
+pytestmark = pytest.mark.gpu
+
+
+@pytest.fixture(scope="module")
+def P():
+    import torch
+
+    if not torch.cuda.is_available():
+        pytest.skip("no CUDA device")
+    import paper_conf_ipps_davistzw17_b200 as pkg
+
+    pkg.lib()
+    return pkg
+
+
+def test_em_recovers_theta(P):
+    n, L = 12, 10000
+    truth, est, single = [], [], []
+    for theta in (0.5, 1.0, 2.0):
+        for rep in range(6):
+            rng = np.random.default_rng(9000 + 100 * rep + int(10 * theta))
+            p, a = synth.coalescent_tree(n, theta, rng)
+            codes = synth.f81_alignment(p, a, L, np.full(4, 0.25), 4 / 3, rng)
+            h = np.sort(a[n:])
+            s_true = 2.0 * sum((n - i) * h[i - 1] for i in range(1, n))
+            ctx = P.Context(synth.to_strings(codes), 0.01, burnin_steps=300, max_proposals=64, max_samples=20000)
+            trace = ctx.mpcgs_em(8, 64, 20000, 31 + rep)
+            truth.append(theta)
+            est.append(trace[-1])
+            single.append(s_true / (n - 1))
+            assert abs(trace[-1] - trace[-3]) <= 0.10 * trace[-1]  # the EM re-drive has settled
+    est, single, truth = map(np.array, (est, single, truth))
+    rel = np.abs(est / single - 1.0)
+    assert np.all(rel <= 0.20) and np.median(rel) <= 0.05, np.c_[truth, single, est]
+    assert np.corrcoef(truth, est)[0, 1] >= 0.75
+    ratio = est / truth
+    assert 0.6 <= ratio.mean() <= 1.6
