@@ -38,22 +38,24 @@ def stale() -> bool:
     return any(os.path.getmtime(p) > t for p in sources() + headers())
 
 
-def build(force: bool = False, verbose: bool = False) -> str:
-    if not force and not stale():
+def build(force: bool = False, verbose: bool = False, out: str = LIB, defines=()) -> str:
+    """Compile libmpcgs.so (or a tuning variant with extra -D defines at `out`)."""
+    if not force and out == LIB and not stale():
         return LIB
     nvcc = os.environ.get("NVCC", "nvcc")
-    tmp = LIB + f".tmp{os.getpid()}"
-    cmd = [nvcc, *NVCC_FLAGS, "-I", INCLUDE, "-I", CSRC, "-o", tmp, *sources(), "-ldl"]
+    tmp = out + f".tmp{os.getpid()}"
+    cmd = [nvcc, *NVCC_FLAGS, *[f"-D{d}" for d in defines], "-I", INCLUDE, "-I", CSRC, "-o", tmp, *sources(), "-ldl"]
     res = subprocess.run(cmd, capture_output=True, text=True)
     if res.returncode != 0:
         sys.stderr.write(res.stdout + res.stderr)
         raise RuntimeError("nvcc failed building libmpcgs.so")
     if verbose:
         sys.stderr.write(res.stderr)
-    with open(os.path.join(PKG, "build_ptxas.log"), "w") as f:
-        f.write(res.stderr)
-    os.replace(tmp, LIB)
-    return LIB
+    if out == LIB:
+        with open(os.path.join(PKG, "build_ptxas.log"), "w") as f:
+            f.write(res.stderr)
+    os.replace(tmp, out)
+    return out
 
 
 if __name__ == "__main__":

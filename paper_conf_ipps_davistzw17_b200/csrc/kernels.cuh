@@ -7,9 +7,18 @@
 namespace mpcgs {
 
 constexpr int PRUNE_THREADS = 128;
-constexpr int PRUNE_SI64 = 2;  // sites interleaved per thread, FP64 partials
-constexpr int PRUNE_SI32 = 2;  // FP32 partials
-constexpr int PRUNE_DR = 4;    // register-resident stack levels (deeper ones spill to shared memory)
+#ifndef MPCGS_SI64
+#define MPCGS_SI64 4
+#endif
+#ifndef MPCGS_SI32
+#define MPCGS_SI32 4
+#endif
+#ifndef MPCGS_DR
+#define MPCGS_DR 3
+#endif
+constexpr int PRUNE_SI64 = MPCGS_SI64;  // sites interleaved per thread, FP64 partials
+constexpr int PRUNE_SI32 = MPCGS_SI32;  // FP32 partials
+constexpr int PRUNE_DR = MPCGS_DR;      // register-resident stack levels (deeper ones spill to shared memory)
 constexpr int PRUNE_SPILL = 2; // shared-memory stack levels; trees needing more use the flat kernel
 
 struct PruneArgs {

@@ -88,11 +88,12 @@ def lib(build_if_missing: bool = True):
     """Load (building if stale) the in-tree libmpcgs.so.  Raises if it cannot."""
     global _lib
     if _lib is None:
-        if build_if_missing and _build.stale():
+        path = os.environ.get("MPCGS_LIB", _build.LIB)  # tuning variants only; default in-tree build
+        if path == _build.LIB and build_if_missing and _build.stale():
             _build.build()
-        if not os.path.exists(_build.LIB):
-            raise MpcgsError(-4, f"CUDA library missing: {_build.LIB}")
-        L = ctypes.CDLL(_build.LIB)
+        if not os.path.exists(path):
+            raise MpcgsError(-4, f"CUDA library missing: {path}")
+        L = ctypes.CDLL(path)
         for name, (res, args) in _SIGS.items():
             f = getattr(L, name)
             f.restype = res
