@@ -209,15 +209,20 @@ def main():
     torch.cuda.set_device(local)
     dist = None
     nccl_id = None
-    if world > 1:
-        import torch.distributed as dist
-
-        dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+    def fresh_nccl_id():  # an ncclUniqueId serves one communicator: make one per context
+        if dist is None:
+            return None
         idb = torch.zeros(128, dtype=torch.uint8, device="cuda")
         if rank == 0:
             idb.copy_(torch.frombuffer(bytearray(P.mpcgs_nccl_unique_id()), dtype=torch.uint8))
         dist.broadcast(idb, 0)
-        nccl_id = bytes(idb.cpu().numpy().tobytes())
+        return bytes(idb.cpu().numpy().tobytes())
+
+    if "WORLD_SIZE" in os.environ:  # launched by torchrun: records all-gathered with NCCL in the library
+        import torch.distributed as dist
+
+        dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+    nccl_id = fresh_nccl_id()
 
     codes = wl["codes"]
     n, L = codes.shape
@@ -272,8 +277,8 @@ def main():
         barrier()
         t0 = time.perf_counter()
         ctx2 = P.Context(rows, wl["theta0"], precision=args.precision, max_proposals=N, max_samples=N * args.steps,
-                         init_tree=(wl["true_parent"], wl["true_age"]), rank=rank, world=world, nccl_id=nccl_id,
-                         stream=stream)
+                         init_tree=(wl["true_parent"], wl["true_age"]), rank=rank, world=world,
+                         nccl_id=fresh_nccl_id(), stream=stream)
         ctx2.mpcgs_sample(N, N * args.steps, wl["chain_seed"] + 1)
         smp = ctx2.mpcgs_get_samples()
         barrier()

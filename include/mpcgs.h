@@ -77,9 +77,12 @@ typedef struct {
     const double* init_age;     /* host [2n-1]; used with init_parent */
     int32_t rank, world;   /* world = 1: one GPU.  world > 1: proposals sharded over ranks */
     const void* nccl_id;   /* host, 128 bytes: ncclUniqueId made by rank 0 with
-                              mpcgs_nccl_unique_id() and broadcast by the caller.  NULL with
-                              world > 1: no communicator; the caller exchanges records itself
-                              (mpcgs_step_local / get_records / put_records / step_finish) */
+                              mpcgs_nccl_unique_id() and broadcast by the caller; the library
+                              then all-gathers the records with NCCL inside mpcgs_sample (also
+                              for world = 1).  NULL with world > 1: no communicator; the caller
+                              exchanges records itself (mpcgs_step_local / get_records /
+                              put_records / step_finish).  An id serves one communicator:
+                              make a fresh one for every context */
     void* stream;          /* cudaStream_t for all work; NULL = the legacy default stream */
     void* workspace;       /* device memory of >= mpcgs_workspace_bytes(...) bytes, 256-B aligned;
                               NULL -> the context allocates (and frees) its own */

@@ -449,7 +449,7 @@ mpcgs_status step_local_launch(mpcgs_ctx* c, uint64_t seed, int64_t step, int N,
 }
 
 mpcgs_status allgather_records(mpcgs_ctx* c, int N) {
-    if (c->world == 1) return MPCGS_OK;
+    if (!c->comm) return MPCGS_OK;  // world = 1 without a communicator
     NcclApi& api = nccl();
     const size_t cnt = (size_t)(N / c->world) * REC;
     double* recv = c->s.rec + REC;  // slot 1
@@ -728,7 +728,7 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
             break;
         }
         if ((st = upload_state(c, parent.data(), age.data()))) break;
-        if (c->world > 1 && cfg->nccl_id) {  // without an id: host-staged record exchange only
+        if (cfg->nccl_id) {  // without an id: no communicator (host-staged exchange when world > 1)
             NcclApi& api = nccl();
             if (!api.ok) { st = fail(c, MPCGS_E_NCCL, "NCCL (libnccl.so.2) could not be loaded"); break; }
             ncclUniqueId id;

@@ -56,3 +56,22 @@ def test_sample_refuses_world_gt1_without_nccl(P):
     with pytest.raises(P.MpcgsError) as ei:
         c.mpcgs_sample(16, 16, 1)
     assert ei.value.status == -3
+
+
+def test_nccl_path_single_rank_matches(P):
+    """The in-library NCCL all-gather path (dlopen'ed NCCL, communicator from an
+    ncclUniqueId, all-gather inside the captured step loop) with one rank gives
+    the same chain as the communicator-free path."""
+    wl = synth.workload("c2", L=500)
+    rows = synth.to_strings(wl["codes"])
+    tree = (wl["true_parent"], wl["true_age"])
+    a = P.Context(rows, wl["theta0"], init_tree=tree, max_proposals=64, max_samples=640, burnin_steps=3)
+    uid = P.mpcgs_nccl_unique_id()
+    assert len(uid) == 128
+    b = P.Context(rows, wl["theta0"], init_tree=tree, max_proposals=64, max_samples=640, burnin_steps=3,
+                  nccl_id=uid)
+    for c in (a, b):
+        c.mpcgs_sample(64, 640, 5)
+    sa, sb = a.mpcgs_get_samples(), b.mpcgs_get_samples()
+    for k in sa:
+        assert np.array_equal(sa[k], sb[k]), k
