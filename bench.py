@@ -168,7 +168,9 @@ def workload_config(args, wl):
     return {"workload": f"{args.workload}: {n} sequences x {L} bp, {wl['N']} proposals/step, theta0 {wl['theta0']}",
             "n_seq": n, "n_sites": L, "proposals_per_step": wl["N"], "theta0": wl["theta0"],
             "precision": args.precision, "l2": "flushed (256 MiB write) between timed steps",
-            "parallelism": f"proposal-sharded x{args.gpus}", "init_tree": "synthetic true tree (ms-style)"}
+            "parallelism": f"proposal-sharded x{args.gpus}", "init_tree": "synthetic true tree (ms-style)",
+            "scoring": "incremental rescoring (f2): partials/s counts the full-pruning equivalent n-1 nodes "
+                       "per proposal and site" if getattr(args, "incremental", False) else "full pruning (5.2.2)"}
 
 
 def main():
@@ -184,6 +186,9 @@ def main():
     ap.add_argument("--precision", type=int, default=64, choices=[32, 64])
     ap.add_argument("--cpu-seconds", type=float, default=12.0)
     ap.add_argument("--no-e2e", action="store_true")
+    ap.add_argument("--no-incremental-block", action="store_true")
+    ap.add_argument("--incremental", action="store_true",
+                    help="score proposals by incremental rescoring (SURVEY 8(f) f2) instead of full pruning")
     args = ap.parse_args()
     args.warmup = max(args.warmup, 3)
 
@@ -238,7 +243,7 @@ def main():
 
     ctx = P.Context(rows, wl["theta0"], precision=args.precision, max_proposals=N, max_samples=N * total_steps,
                     init_tree=(wl["true_parent"], wl["true_age"]), rank=rank, world=world, nccl_id=nccl_id,
-                    stream=stream)
+                    stream=stream, incremental=args.incremental)
     # warm-up (untimed): W steps
     ctx.mpcgs_sample(N, N * args.warmup, wl["chain_seed"])
     ctx.mpcgs_set_timing(3)   # per-step + per-prune CUDA events, L2 flush between steps
@@ -278,7 +283,7 @@ def main():
         t0 = time.perf_counter()
         ctx2 = P.Context(rows, wl["theta0"], precision=args.precision, max_proposals=N, max_samples=N * args.steps,
                          init_tree=(wl["true_parent"], wl["true_age"]), rank=rank, world=world,
-                         nccl_id=fresh_nccl_id(), stream=stream)
+                         nccl_id=fresh_nccl_id(), stream=stream, incremental=args.incremental)
         ctx2.mpcgs_sample(N, N * args.steps, wl["chain_seed"] + 1)
         smp = ctx2.mpcgs_get_samples()
         barrier()
@@ -294,6 +299,28 @@ def main():
                "d2h_bytes_per_step": d2h / args.steps, "includes": "init (alignment H2D, G0 scoring) + sampling + "
                "sample D2H, wall clock"}
 
+    # the same workload scored by incremental rescoring, reported
+    # beside the full-pruning headline (its partials/s counts n-1 nodes per proposal)
+    incr = None
+    if not args.incremental and not args.no_incremental_block:
+        ctx3 = P.Context(rows, wl["theta0"], precision=args.precision, max_proposals=N,
+                         max_samples=N * (args.warmup + args.steps), init_tree=(wl["true_parent"], wl["true_age"]),
+                         rank=rank, world=world, nccl_id=fresh_nccl_id(), stream=stream, incremental=True)
+        ctx3.mpcgs_sample(N, N * args.warmup, wl["chain_seed"])
+        ctx3.mpcgs_set_timing(3)
+        barrier()
+        ctx3.mpcgs_sample(N, N * args.steps, wl["chain_seed"] + 1)
+        barrier()
+        l3, s3, _ = ctx3.mpcgs_last_timing()
+        t3 = torch.tensor([l3, s3], dtype=torch.float64, device="cuda")
+        if dist is not None:
+            dist.all_reduce(t3, op=dist.ReduceOp.MAX)
+        l3, s3 = float(t3[0]), float(t3[1])
+        ctx3.free()
+        incr = {"proposals_per_s": N * args.steps / (l3 / 1e3), "ms_per_step": l3 / args.steps,
+                "partials_equiv_per_s": partials / (l3 / 1e3), "score_kernel_share": s3 / l3,
+                "speedup_vs_full": loop_ms / l3, "kernel": "k_score_incr"}
+
     cpu = None
     if rank == 0 and world == 1 and args.cpu_seconds > 0:
         v, st, dt = cpu_oracle_sample(wl, args.cpu_seconds)
@@ -307,6 +334,7 @@ def main():
             "vs_baseline": None, "dtype": "f64" if args.precision == 64 else "f32", "data": "synthetic",
             "config": workload_config(args, wl), "proposals_per_s": N * args.steps / (loop_ms / 1e3),
             "roofline": roof, "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": int(launches),
+            "incremental_rescoring": incr,
             "clocks": clocks,
         }
         print(json.dumps(line), flush=True)

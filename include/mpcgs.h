@@ -87,15 +87,22 @@ typedef struct {
     void* workspace;       /* device memory of >= mpcgs_workspace_bytes(...) bytes, 256-B aligned;
                               NULL -> the context allocates (and frees) its own */
     size_t workspace_bytes;
+    int32_t incremental;   /* 0: every proposal is scored by full pruning (the paper, 5.2.2).
+                              1: incremental rescoring: the generator's partials
+                              of all nodes and sites stay in device memory and a proposal
+                              recomputes only T, Par and the ancestors of Par (L1390-1398) */
 } mpcgs_config;
 
 /* [host-only] Fill cfg with defaults: empirical pi, default u, precision 64, burn-in 0,
  * max_proposals 1024, max_samples 1<<20, world 1. */
 void mpcgs_config_default(mpcgs_config* cfg);
 
-/* [host-only] Device bytes a context needs for these capacities. */
+/* [host-only] Device bytes a context needs for these capacities (full pruning). */
 size_t mpcgs_workspace_bytes(int32_t n_seq, int32_t n_sites, int32_t max_proposals,
                              int64_t max_samples, int32_t precision);
+/* [host-only] Same, with incremental rescoring on (incremental != 0). */
+size_t mpcgs_workspace_bytes_ex(int32_t n_seq, int32_t n_sites, int32_t max_proposals,
+                                int64_t max_samples, int32_t precision, int32_t incremental);
 
 /* Create a context: validate and copy the alignment, compute pi and u, build G0
  * (init_parent/init_age, else UPGMA), upload everything to the device and score

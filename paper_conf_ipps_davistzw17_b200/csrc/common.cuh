@@ -177,6 +177,20 @@ struct DevState {
     double* theta_buf;
     int Nmax, tiles_max;
     int64_t Mmax;
+    // incremental rescoring: the generator's partial likelihood
+    // of every interior node at every site, and what each proposal changed
+    int incremental;
+    void* GL;           // [n-1][Lg][4] partials of interior node v at [v-n] (float or double)
+    int32_t* GE;        // [n-1][Lg] power-of-two exponent removed from GL (whole subtree)
+    int Lg;             // site stride of GL / GE
+    int32_t* path;      // [n] ancestors of Par: A, parent(A), ..., root (context)
+    int32_t* pathsib;   // [n] the other child of each ancestor
+    int32_t* ixyz;      // [Nmax][4] per local proposal: pair children x, y and third child z
+    double* iee;        // [Nmax][10] e/em of the changed branches x, y, z, T, Par
+    int32_t* cinfo;     // committed step: T, Par, I (drawn slot), d, rootcase
+    int32_t* cpath;     // [n] committed step's ancestor path
+    int32_t* csib;      // [n]
+    int32_t* gen_order; // [n-1] interior nodes children-first (full partial recompute)
 };
 
 // counters[2] status bits

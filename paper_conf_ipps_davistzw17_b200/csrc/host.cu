@@ -59,6 +59,7 @@ struct mpcgs_ctx {
     DevState s{};
     int n = 0, L = 0, nn = 0, Lpad = 0, nops = 0, depth = 0, precision = 64;
     int world = 1, rank = 0, burnin = 0;
+    bool incremental = false;
     int Nmax = 0;
     int64_t Mmax = 0;
     double theta0 = 0.0, sample_theta0 = 0.0;
@@ -111,7 +112,7 @@ mpcgs_status fail(mpcgs_ctx* c, mpcgs_status st, const std::string& msg) {
 struct Layout {
     size_t codes, codes2, parent, left, right, need, age, e, em, gen, ctx_i, ctx_d, tau, len, lcnt, entry, omega, fixed;
     size_t tree_need, rec, sched_op, sched_e, tile_part, tile_cnt, sS, sL, sStep, sSlot, counters, last_draws, theta_buf,
-        theta_cnt, score_out, total;
+        theta_cnt, score_out, GL, GE, path, pathsib, cpath, csib, ixyz, iee, cinfo, gen_order, total;
     int tiles_max;
 };
 
@@ -120,7 +121,7 @@ size_t al(size_t x) { return (x + 255) & ~(size_t)255; }
 // 2-bit packed tip codes, 16 sites per 32-bit word, rows padded past the last tile
 int codes2_words(int L) { return ((L + 4096 + 63) / 64) * 4; }
 
-Layout layout(int n, int L, int Nmax, int64_t Mmax, int precision) {
+Layout layout(int n, int L, int Nmax, int64_t Mmax, int precision, int incremental = 0) {
     Layout y{};
     const int nn = 2 * n - 1, nops = n - 1;
     const int Lpad = (L + 15) & ~15;
@@ -165,6 +166,17 @@ Layout layout(int n, int L, int Nmax, int64_t Mmax, int precision) {
     y.theta_buf = take(8 * (size_t)(2 * MPCGS_MAX_GRID + 3 * 296 + 16));
     y.theta_cnt = take(16);
     y.score_out = take(8 * (size_t)Nmax);
+    const size_t tsz = precision == 32 ? 4 : 8;
+    y.GL = take(incremental ? 4 * tsz * (size_t)(n - 1) * Lpad : 0);
+    y.GE = take(incremental ? 4 * (size_t)(n - 1) * Lpad : 0);
+    y.path = take(4 * (size_t)n);
+    y.pathsib = take(4 * (size_t)n);
+    y.cpath = take(4 * (size_t)n);
+    y.csib = take(4 * (size_t)n);
+    y.ixyz = take(16 * (size_t)Nmax);
+    y.iee = take(80 * (size_t)Nmax);
+    y.cinfo = take(32);
+    y.gen_order = take(4 * (size_t)n);
     y.total = o;
     return y;
 }
@@ -421,6 +433,26 @@ mpcgs_status upload_state(mpcgs_ctx* c, const int32_t* parent, const double* age
     CU(cudaMemcpyAsync(c->s.e, ht.e.data(), 8 * (size_t)nn, cudaMemcpyHostToDevice, c->work));
     CU(cudaMemcpyAsync(c->s.em, ht.em.data(), 8 * (size_t)nn, cudaMemcpyHostToDevice, c->work));
     CU(cudaMemcpyAsync(c->s.gen, gen, 16, cudaMemcpyHostToDevice, c->work));
+    if (c->incremental) {
+        // interior nodes children-first (post-order), then every node's partials
+        std::vector<int32_t> order;
+        std::vector<int> st{ht.root};
+        std::vector<char> done(nn, 0);
+        while (!st.empty()) {
+            const int v = st.back();
+            const int a = ht.left[v], b2 = ht.right[v];
+            if ((a >= n && !done[a]) || (b2 >= n && !done[b2])) {
+                if (a >= n && !done[a]) st.push_back(a);
+                if (b2 >= n && !done[b2]) st.push_back(b2);
+                continue;
+            }
+            done[v] = 1;
+            order.push_back(v);
+            st.pop_back();
+        }
+        CU(cudaMemcpyAsync(c->s.gen_order, order.data(), 4 * order.size(), cudaMemcpyHostToDevice, c->work));
+        CU(launch_gen_partials(c->s, c->work));
+    }
     CU(cudaStreamSynchronize(c->work));
     return MPCGS_OK;
 }
@@ -441,8 +473,21 @@ mpcgs_status step_local_launch(mpcgs_ctx* c, uint64_t seed, int64_t step, int N,
     CU(launch_propose(c->s, seed, step, first, count, c->work));
     PruneArgs a = prune_args(c, N, c->s.rec, first, REC);
     if (pre) CU(cudaEventRecord(pre, c->work));
-    int np = 0;
-    CU(launch_prune(a, count, c->depth, c->precision, c->work, &np));
+    int np = 1;
+    if (c->incremental) {
+        IncrArgs ia{};
+        ia.count = count;
+        ia.tiles = a.tiles;
+        ia.sites_per_cta = a.sites_per_cta;
+        ia.tile_part = c->s.tile_part;
+        ia.tile_cnt = c->s.tile_cnt;
+        ia.out = c->s.rec;
+        ia.out_first = first;
+        ia.out_stride = REC;
+        CU(launch_score_incr(c->s, ia, c->work));
+    } else {
+        CU(launch_prune(a, count, c->depth, c->precision, c->work, &np));
+    }
     if (post) CU(cudaEventRecord(post, c->work));
     c->launches += (with_context ? 2 : 1) + np;
     return MPCGS_OK;
@@ -480,8 +525,13 @@ void mpcgs_config_default(mpcgs_config* cfg) {
 
 size_t mpcgs_workspace_bytes(int32_t n_seq, int32_t n_sites, int32_t max_proposals, int64_t max_samples,
                              int32_t precision) {
+    return mpcgs_workspace_bytes_ex(n_seq, n_sites, max_proposals, max_samples, precision, 0);
+}
+
+size_t mpcgs_workspace_bytes_ex(int32_t n_seq, int32_t n_sites, int32_t max_proposals, int64_t max_samples,
+                                int32_t precision, int32_t incremental) {
     if (n_seq < 2 || n_sites < 1 || max_proposals < 1 || max_samples < 0) return 0;
-    return layout(n_seq, n_sites, max_proposals, max_samples, precision).total;
+    return layout(n_seq, n_sites, max_proposals, max_samples, precision, incremental != 0).total;
 }
 
 void mpcgs_philox(const uint32_t ctr[4], const uint32_t key[2], uint32_t out[4]) {
@@ -647,7 +697,8 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
         upgma(n, L, codes.data(), theta0, parent.data(), age.data());
     }
     // device memory
-    Layout y = layout(n, L, c->Nmax, c->Mmax, c->precision);
+    c->incremental = cfg->incremental != 0;
+    Layout y = layout(n, L, c->Nmax, c->Mmax, c->precision, c->incremental);
     mpcgs_status st = MPCGS_OK;
     do {
         if (cudaStreamCreateWithFlags(&c->work, cudaStreamNonBlocking) != cudaSuccess ||
@@ -709,6 +760,18 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
         s.theta_buf = (double*)(b + y.theta_buf);
         s.Nmax = c->Nmax;
         s.tiles_max = y.tiles_max;
+        s.incremental = c->incremental ? 1 : 0;
+        s.GL = c->incremental ? (void*)(b + y.GL) : nullptr;
+        s.GE = c->incremental ? (int32_t*)(b + y.GE) : nullptr;
+        s.Lg = c->Lpad;
+        s.path = (int32_t*)(b + y.path);
+        s.pathsib = (int32_t*)(b + y.pathsib);
+        s.cpath = (int32_t*)(b + y.cpath);
+        s.csib = (int32_t*)(b + y.csib);
+        s.ixyz = (int32_t*)(b + y.ixyz);
+        s.iee = (double*)(b + y.iee);
+        s.cinfo = (int32_t*)(b + y.cinfo);
+        s.gen_order = (int32_t*)(b + y.gen_order);
         s.Mmax = c->Mmax;
         c->theta_cnt = (unsigned*)(b + y.theta_cnt);
         c->score_out = (double*)(b + y.score_out);
@@ -788,6 +851,10 @@ mpcgs_status mpcgs_sample(mpcgs_ctx* c, int32_t N, int64_t M, uint64_t seed) {
         if ((s2 = allgather_records(c, N))) return s2;
         CU(launch_draw(c->s, seed, -1, N, -1, c->burnin, M, steps, c->work));
         ++c->launches;
+        if (c->incremental) {
+            CU(launch_commit_incr(c->s, c->work));
+            ++c->launches;
+        }
         return MPCGS_OK;
     };
     if (c->timing & 1) {
@@ -811,6 +878,10 @@ mpcgs_status mpcgs_sample(mpcgs_ctx* c, int32_t N, int64_t M, uint64_t seed) {
             if ((st = allgather_records(c, N))) return st;
             CU(launch_draw(c->s, seed, -1, N, -1, c->burnin, M, steps, c->work));
             ++c->launches;
+            if (c->incremental) {
+                CU(launch_commit_incr(c->s, c->work));
+                ++c->launches;
+            }
             CU(cudaEventRecord(c->evpool[4 * k + 3], c->work));
         }
         CU(cudaEventSynchronize(c->evpool[4 * (steps - 1) + 3]));
@@ -963,6 +1034,7 @@ mpcgs_status mpcgs_step_finish(mpcgs_ctx* c, int64_t step, int32_t N, int32_t K,
     if (st) return st;
     CU(cudaMemsetAsync(c->s.counters + 2, 0, 8, c->work));
     CU(launch_draw(c->s, seed, step, N, K, 0, 0, 0, c->work));
+    if (c->incremental) CU(launch_commit_incr(c->s, c->work));
     if (draws) CU(cudaMemcpyAsync(draws, c->s.last_draws, 4 * (size_t)K, cudaMemcpyDeviceToHost, c->work));
     if ((st = leave(c))) return st;
     return check_status(c);
@@ -978,6 +1050,7 @@ mpcgs_status mpcgs_step_trace(mpcgs_ctx* c, int64_t step, int32_t N, int32_t K, 
     CU(cudaMemsetAsync(c->s.counters + 2, 0, 8, c->work));
     if ((st = step_local_launch(c, seed, step, N))) return st;
     CU(launch_draw(c->s, seed, step, N, K, 0, 0, 0, c->work));
+    if (c->incremental) CU(launch_commit_incr(c->s, c->work));
     std::vector<double> rec((size_t)(N + 1) * REC);
     int32_t ci[16];
     CU(cudaMemcpyAsync(rec.data(), c->s.rec, rec.size() * 8, cudaMemcpyDeviceToHost, c->work));

@@ -1,0 +1,264 @@
+// incr.cu -- incremental rescoring (the alternative the paper
+// weighed and rejected for Kepler, 5.2.2 L1390-1398).
+//
+// The generator's partial likelihood vector of every interior node at every
+// site (Eq. 19) is kept in HBM (GL, with its power-of-two exponent GE).  A
+// LAMARC proposal changes only the two resimulated nodes (T, Par) and the
+// branch above Par, so its root partial is
+//     v_T  = br(L_x) (.) br(L_y),   v_Par = br(v_T) (.) br(L_z),
+//     v_a  = br(v_prev) (.) br(L_sib(a))   for a = A, parent(A), ..., root,
+// with L_x, L_y, L_z, L_sib(a) read from GL (or tip indicators).  The work per
+// proposal and site falls from n-1 nodes to 2 + depth(A) nodes.  After each
+// draw k_commit_incr rewrites the changed nodes of the new generator.
+// Results equal full pruning up to FP rounding order.
+#include "arith.cuh"
+#include "common.cuh"
+#include "kernels.cuh"
+
+namespace mpcgs {
+
+constexpr int INCR_THREADS = 128;
+constexpr int INCR_PG = 8;  // proposals per CTA (per-thread accumulators)
+
+// node c at `site`: tip -> indicator vector, exponent 0; interior -> GL, GE
+template <typename T>
+__device__ __forceinline__ int load_node(const DevState& s, int c, int site, T (&v)[4]) {
+    if (c < s.n) {
+        const int x = __ldg(s.codes + (size_t)c * s.Lpad + site);
+        v[0] = x == 0 ? T(1) : T(0);
+        v[1] = x == 1 ? T(1) : T(0);
+        v[2] = x == 2 ? T(1) : T(0);
+        v[3] = x == 3 ? T(1) : T(0);
+        return 0;
+    }
+    const size_t i = (size_t)(c - s.n) * s.Lg + site;
+    ld4<T>(v, reinterpret_cast<const T*>(s.GL) + 4 * i);
+    return s.GE[i];
+}
+
+template <typename T>
+__device__ __forceinline__ void store_node(const DevState& s, int v, int site, const T (&x)[4], int e) {
+    const size_t i = (size_t)(v - s.n) * s.Lg + site;
+    T* g = reinterpret_cast<T*>(s.GL) + 4 * i;
+    g[0] = x[0]; g[1] = x[1]; g[2] = x[2]; g[3] = x[3];
+    s.GE[i] = e;
+}
+
+// v = br(a, ea) (.) br(b, eb), exponent ka + kb (+ own rescale)
+template <typename T>
+__device__ __forceinline__ int combine(T (&a)[4], int ka, T ea, T ema, T (&b)[4], int kb, T eb, T emb,
+                                      const T (&pi)[4]) {
+    branch<T>(a, ea, ema, pi);
+    branch<T>(b, eb, emb, pi);
+#pragma unroll
+    for (int i = 0; i < 4; ++i) a[i] *= b[i];
+    const int k = rescale_k(a);
+    if (k) {
+        const T f = pow2(k, T(0));
+        a[0] *= f; a[1] *= f; a[2] *= f; a[3] *= f;
+    }
+    return ka + kb + k;
+}
+
+// ---------------------------------------------------------------- full generator partials
+template <typename T>
+__global__ void __launch_bounds__(256) k_gen_partials(DevState s) {
+    const int site = blockIdx.x * blockDim.x + threadIdx.x;
+    if (site >= s.L) return;
+    const T pi[4] = {(T)s.pi[0], (T)s.pi[1], (T)s.pi[2], (T)s.pi[3]};
+    for (int i = 0; i < s.n - 1; ++i) {  // children before parents
+        const int v = s.gen_order[i];
+        const int l = s.left[v], r = s.right[v];
+        T a[4], b[4];
+        const int ka = load_node<T>(s, l, site, a);
+        const int kb = load_node<T>(s, r, site, b);
+        const int k = combine<T>(a, ka, (T)s.e[l], (T)s.em[l], b, kb, (T)s.e[r], (T)s.em[r], pi);
+        store_node<T>(s, v, site, a, k);
+    }
+}
+
+// ---------------------------------------------------------------- commit of the drawn proposal
+template <typename T>
+__global__ void __launch_bounds__(256) k_commit_incr(DevState s) {
+    const int site = blockIdx.x * blockDim.x + threadIdx.x;
+    const int I = s.cinfo[2];
+    if (I <= 0 || site >= s.L) return;  // the generator was kept: nothing changed
+    const T pi[4] = {(T)s.pi[0], (T)s.pi[1], (T)s.pi[2], (T)s.pi[3]};
+    const int Tn = s.cinfo[0], Par = s.cinfo[1], d = s.cinfo[3];
+    T cur[4], b[4];
+    int l = s.left[Tn], r = s.right[Tn];
+    int kc = load_node<T>(s, l, site, cur);
+    int kb = load_node<T>(s, r, site, b);
+    kc = combine<T>(cur, kc, (T)s.e[l], (T)s.em[l], b, kb, (T)s.e[r], (T)s.em[r], pi);
+    store_node<T>(s, Tn, site, cur, kc);
+    const int z = s.left[Par] == Tn ? s.right[Par] : s.left[Par];
+    kb = load_node<T>(s, z, site, b);
+    kc = combine<T>(cur, kc, (T)s.e[Tn], (T)s.em[Tn], b, kb, (T)s.e[z], (T)s.em[z], pi);
+    store_node<T>(s, Par, site, cur, kc);
+    int prev = Par;
+    for (int i = 0; i < d; ++i) {
+        const int a = s.cpath[i], sib = s.csib[i];
+        kb = load_node<T>(s, sib, site, b);
+        kc = combine<T>(cur, kc, (T)s.e[prev], (T)s.em[prev], b, kb, (T)s.e[sib], (T)s.em[sib], pi);
+        store_node<T>(s, a, site, cur, kc);
+        prev = a;
+    }
+}
+
+// ---------------------------------------------------------------- proposal scores
+// Grid (site tiles, ceil(count / INCR_PG)); each CTA scores INCR_PG proposals of
+// this rank over one tile.  Per site the three children's partials are loaded
+// once and reused by every proposal of the CTA.
+template <typename T>
+__global__ void __launch_bounds__(INCR_THREADS) k_score_incr(DevState s, IncrArgs a) {
+    __shared__ int sh_path[128], sh_sib[128];
+    __shared__ double sh_pe[4 * 128];   // e, em of the path branches and of the siblings' branches
+    __shared__ int sh_xyz[INCR_PG][4];
+    __shared__ double sh_ee[INCR_PG][10];
+    __shared__ double s_red[INCR_THREADS / 32];
+    __shared__ bool s_last;
+    const int tid = threadIdx.x, tile = blockIdx.x;
+    const int p0 = blockIdx.y * INCR_PG;
+    const int np = min(INCR_PG, a.count - p0);
+    const int c0 = s.ctx_i[6], c1 = s.ctx_i[7], c2 = s.ctx_i[8];
+    const bool rootcase = s.ctx_i[3] != 0;
+    const int d = s.ctx_i[11];
+    const int dc = min(d, 128);  // ancestors whose ids / factors are cached in shared memory
+    for (int i = tid; i < dc; i += INCR_THREADS) {
+        const int an = s.path[i], sb = s.pathsib[i];
+        sh_path[i] = an;
+        sh_sib[i] = sb;
+        sh_pe[4 * i + 0] = s.e[an];
+        sh_pe[4 * i + 1] = s.em[an];
+        sh_pe[4 * i + 2] = s.e[sb];
+        sh_pe[4 * i + 3] = s.em[sb];
+    }
+    for (int i = tid; i < np * 4; i += INCR_THREADS) sh_xyz[i >> 2][i & 3] = s.ixyz[4 * (p0 + (i >> 2)) + (i & 3)];
+    for (int i = tid; i < np * 10; i += INCR_THREADS) sh_ee[i / 10][i % 10] = s.iee[10 * (p0 + i / 10) + i % 10];
+    __syncthreads();
+    const T pi[4] = {(T)s.pi[0], (T)s.pi[1], (T)s.pi[2], (T)s.pi[3]};
+    const int s_begin = tile * a.sites_per_cta;
+    const int s_end = min(s.L, s_begin + a.sites_per_cta);
+    double mant[INCR_PG];
+    int expo[INCR_PG];
+#pragma unroll
+    for (int j = 0; j < INCR_PG; ++j) {
+        mant[j] = 1.0;
+        expo[j] = 0;
+    }
+    for (int site = s_begin + tid; site < s_end; site += INCR_THREADS) {
+        T L0[4], L1[4], L2[4];
+        const int k0 = load_node<T>(s, c0, site, L0);
+        const int k1 = load_node<T>(s, c1, site, L1);
+        const int k2 = load_node<T>(s, c2, site, L2);
+#pragma unroll
+        for (int j = 0; j < INCR_PG; ++j) {
+            if (j >= np) break;
+            const int x = sh_xyz[j][0], y = sh_xyz[j][1];
+            const double* ee = sh_ee[j];
+            T vx[4], vy[4], vz[4];
+            int kx, ky, kz;
+            // pair code 0 = (c1,c2) | c3, 1 = (c1,c3) | c2, 2 = (c2,c3) | c1 (S14)
+            if (x == c0 && y == c1) {
+#pragma unroll
+                for (int i = 0; i < 4; ++i) { vx[i] = L0[i]; vy[i] = L1[i]; vz[i] = L2[i]; }
+                kx = k0; ky = k1; kz = k2;
+            } else if (x == c0) {
+#pragma unroll
+                for (int i = 0; i < 4; ++i) { vx[i] = L0[i]; vy[i] = L2[i]; vz[i] = L1[i]; }
+                kx = k0; ky = k2; kz = k1;
+            } else {
+#pragma unroll
+                for (int i = 0; i < 4; ++i) { vx[i] = L1[i]; vy[i] = L2[i]; vz[i] = L0[i]; }
+                kx = k1; ky = k2; kz = k0;
+            }
+            int kc = combine<T>(vx, kx, (T)ee[0], (T)ee[1], vy, ky, (T)ee[2], (T)ee[3], pi);   // T
+            kc = combine<T>(vx, kc, (T)ee[6], (T)ee[7], vz, kz, (T)ee[4], (T)ee[5], pi);         // Par
+            if (!rootcase) {
+                T pe = (T)ee[8], pem = (T)ee[9];  // branch Par -> A
+                for (int i = 0; i < d; ++i) {
+                    int sb;
+                    T se, sem, ae, aem;
+                    if (i < dc) {
+                        sb = sh_sib[i];
+                        ae = (T)sh_pe[4 * i + 0]; aem = (T)sh_pe[4 * i + 1];
+                        se = (T)sh_pe[4 * i + 2]; sem = (T)sh_pe[4 * i + 3];
+                    } else {
+                        const int an = s.path[i];
+                        sb = s.pathsib[i];
+                        ae = (T)s.e[an]; aem = (T)s.em[an]; se = (T)s.e[sb]; sem = (T)s.em[sb];
+                    }
+                    T vs[4];
+                    const int ks = load_node<T>(s, sb, site, vs);
+                    kc = combine<T>(vx, kc, pe, pem, vs, ks, se, sem, pi);
+                    pe = ae;
+                    pem = aem;
+                }
+            }
+            // Eq. 21 at the root, multiplied into this proposal's accumulator
+            T ls = pi[0] * vx[0];
+            ls = fma(pi[1], vx[1], ls);
+            ls = fma(pi[2], vx[2], ls);
+            ls = fma(pi[3], vx[3], ls);
+            mant[j] *= (double)ls;
+            const int hi = __double2hiint(mant[j]);
+            const int ex = ((hi >> 20) & 2047) - 1023;
+            if (ex > -1023) {
+                mant[j] = __hiloint2double((hi & 0x800FFFFF) | (1023 << 20), __double2loint(mant[j]));
+                expo[j] += ex;
+            }
+            expo[j] -= kc;
+        }
+    }
+    for (int j = 0; j < np; ++j) {
+        double ll = (mant[j] > 0.0) ? log(mant[j]) + (double)expo[j] * 0.69314718055994530942 : -INFINITY;
+#pragma unroll
+        for (int off = 16; off > 0; off >>= 1) ll += __shfl_down_sync(0xffffffffu, ll, off);
+        if ((tid & 31) == 0) s_red[tid >> 5] = ll;
+        __syncthreads();
+        if (tid == 0) {
+            double t = 0.0;
+            for (int w = 0; w < INCR_THREADS / 32; ++w) t += s_red[w];
+            const int tree = p0 + j;
+            a.tile_part[(size_t)tree * a.tiles + tile] = t;
+            __threadfence();
+            const unsigned prev = atomicAdd(a.tile_cnt + tree, 1u);
+            s_last = (prev == (unsigned)(a.tiles - 1));
+        }
+        __syncthreads();
+        if (s_last && tid == 0) {
+            __threadfence();
+            const int tree = p0 + j;
+            double t = 0.0;
+            const volatile double* tp = a.tile_part + (size_t)tree * a.tiles;
+            for (int k = 0; k < a.tiles; ++k) t += tp[k];
+            a.out[(size_t)(a.out_first + tree) * a.out_stride] = t;
+            a.tile_cnt[tree] = 0u;
+        }
+        __syncthreads();
+    }
+}
+
+cudaError_t launch_gen_partials(const DevState& s, cudaStream_t st) {
+    const int blocks = (s.L + 255) / 256;
+    if (s.precision == 32) k_gen_partials<float><<<blocks, 256, 0, st>>>(s);
+    else k_gen_partials<double><<<blocks, 256, 0, st>>>(s);
+    return cudaGetLastError();
+}
+
+cudaError_t launch_commit_incr(const DevState& s, cudaStream_t st) {
+    const int blocks = (s.L + 255) / 256;
+    if (s.precision == 32) k_commit_incr<float><<<blocks, 256, 0, st>>>(s);
+    else k_commit_incr<double><<<blocks, 256, 0, st>>>(s);
+    return cudaGetLastError();
+}
+
+cudaError_t launch_score_incr(const DevState& s, const IncrArgs& a, cudaStream_t st) {
+    if (a.count <= 0) return cudaSuccess;
+    dim3 grid(a.tiles, (a.count + INCR_PG - 1) / INCR_PG);
+    if (s.precision == 32) k_score_incr<float><<<grid, INCR_THREADS, 0, st>>>(s, a);
+    else k_score_incr<double><<<grid, INCR_THREADS, 0, st>>>(s, a);
+    return cudaGetLastError();
+}
+
+}  // namespace mpcgs

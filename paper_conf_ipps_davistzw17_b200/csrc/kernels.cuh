@@ -55,6 +55,19 @@ cudaError_t launch_draw(const DevState& s, uint64_t seed, int64_t step, int N, i
                         int64_t M, int64_t total_steps, cudaStream_t st);
 cudaError_t launch_fill_gen_record(const DevState& s, cudaStream_t st);
 
+// incremental rescoring (incr.cu)
+struct IncrArgs {
+    int count;                 // proposals of this rank (local slots 0..count-1)
+    int tiles, sites_per_cta;
+    double* tile_part;         // [count][tiles]
+    uint32_t* tile_cnt;        // [count]
+    double* out;               // logL of local proposal t -> out[(out_first + t) * out_stride]
+    int out_first, out_stride;
+};
+cudaError_t launch_gen_partials(const DevState& s, cudaStream_t st);
+cudaError_t launch_commit_incr(const DevState& s, cudaStream_t st);
+cudaError_t launch_score_incr(const DevState& s, const IncrArgs& a, cudaStream_t st);
+
 // theta kernels (theta.cu)
 cudaError_t launch_minmax(const double* S, int64_t M, double* out2, cudaStream_t st);
 cudaError_t launch_theta_grid(const double* S, int64_t M, int n, double theta0, double lo, double hi, int G,

@@ -265,6 +265,16 @@ __device__ void context_body(const DevState& s, uint64_t seed, int64_t step_arg,
         s.ctx_i[10] = sh[10];
         for (int i = 0; i < 4; ++i) s.ctx_d[i] = shd[i];
         s.counters[4] = T;
+        if (s.incremental) {  // ancestors of Par and their other children (f2)
+            int d = 0, prev = Par;
+            for (int a = sh[2]; a >= 0; a = s.parent[a]) {
+                s.path[d] = a;
+                s.pathsib[d] = s.left[a] == prev ? s.right[a] : s.left[a];
+                prev = a;
+                ++d;
+            }
+            s.ctx_i[11] = d;
+        }
     }
 }
 
@@ -571,6 +581,13 @@ __global__ void __launch_bounds__(32) k_propose(DevState s, uint64_t seed, int64
             else if (c == Par) { e = sh_e2[2]; em = sh_e2[3]; }
             else { e = ge[c]; em = gem[c]; }
         };
+        if (s.incremental) {
+            int32_t* q = s.ixyz + 4 * (size_t)local;
+            q[0] = x; q[1] = y; q[2] = z; q[3] = 0;
+            double* ee = s.iee + 10 * (size_t)local;
+            for (int i = 0; i < 6; ++i) ee[i] = sh_d[2 + i];
+            for (int i = 0; i < 4; ++i) ee[6 + i] = sh_e2[i];
+        }
         uint32_t* op_out = s.sched_op + (size_t)local * s.nops;
         E4* e_out = reinterpret_cast<E4*>(s.sched_e) + (size_t)local * s.nops;
         emit_schedule(
@@ -772,6 +789,11 @@ __global__ void __launch_bounds__(DRAW_THREADS) k_draw(DevState s, uint64_t seed
             if (s_store) s.counters[1] = stored + K;
         }
         s.counters[3] = K;
+    }
+    if (tid == 0 && s.incremental) {  // what the partials update (k_commit_incr) needs
+        const int d = s.ctx_i[11];
+        s.cinfo[0] = T; s.cinfo[1] = Par; s.cinfo[2] = I; s.cinfo[3] = d; s.cinfo[4] = s.ctx_i[3];
+        for (int i = 0; i < d; ++i) { s.cpath[i] = s.path[i]; s.csib[i] = s.pathsib[i]; }
     }
     // device loop: the next step's context, from the committed generator
     if (K_arg < 0 && step + 1 < total_steps) {

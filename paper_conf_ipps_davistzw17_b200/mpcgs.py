@@ -38,7 +38,7 @@ class mpcgs_config(ctypes.Structure):
         ("max_samples", ctypes.c_int64), ("init_parent", ctypes.c_void_p),
         ("init_age", ctypes.c_void_p), ("rank", ctypes.c_int32), ("world", ctypes.c_int32),
         ("nccl_id", ctypes.c_void_p), ("stream", ctypes.c_void_p), ("workspace", ctypes.c_void_p),
-        ("workspace_bytes", ctypes.c_size_t),
+        ("workspace_bytes", ctypes.c_size_t), ("incremental", ctypes.c_int32),
     ]
 
 
@@ -50,6 +50,7 @@ _i32, _i64, _u64, _f64, _sz = ctypes.c_int32, ctypes.c_int64, ctypes.c_uint64, c
 _SIGS = {
     "mpcgs_config_default": (None, [_P]),
     "mpcgs_workspace_bytes": (_sz, [_i32, _i32, _i32, _i64, _i32]),
+    "mpcgs_workspace_bytes_ex": (_sz, [_i32, _i32, _i32, _i64, _i32, _i32]),
     "mpcgs_init": (_i32, [_P, _P, _f64, _P]),
     "mpcgs_init_phylip": (_i32, [ctypes.c_char_p, _P, _f64, _P]),
     "mpcgs_sample": (_i32, [_P, _i32, _i64, _u64]),
@@ -195,7 +196,7 @@ class Context:
 
     def __init__(self, rows, theta0, *, precision=64, burnin_steps=0, max_proposals=1024,
                  max_samples=1 << 20, base_freq=None, mu=0.0, init_tree=None, rank=0, world=1,
-                 nccl_id=None, stream=None, workspace=None, phylip=None):
+                 nccl_id=None, stream=None, workspace=None, phylip=None, incremental=False):
         L = lib()
         cfg = mpcgs_config()
         L.mpcgs_config_default(ctypes.byref(cfg))
@@ -207,6 +208,7 @@ class Context:
         cfg.burnin_steps = int(burnin_steps)
         cfg.max_proposals = int(max_proposals)
         cfg.max_samples = int(max_samples)
+        cfg.incremental = int(bool(incremental))
         self._keep = []
         if init_tree is not None:
             p = _i32a(init_tree[0])

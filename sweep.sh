@@ -1,7 +1,7 @@
 #!/bin/bash
 # bench sweep over the BASELINE.json configs (1 GPU); one JSON line per point
 OUT=gpurun_out/sweep_${1:-x}.jsonl; : > $OUT
-run() { timeout 300 python bench.py --cpu-seconds 0 --no-e2e --steps ${STEPS:-10} --warmup 3 "$@" 2>/dev/null | tail -1 >> $OUT; }
+run() { timeout 300 python bench.py --cpu-seconds 0 --no-e2e --no-incremental-block --steps ${STEPS:-10} --warmup 3 "$@" 2>/dev/null | tail -1 >> $OUT; }
 run --workload c1
 run --workload c2
 run --workload c3

@@ -95,14 +95,15 @@ def test_underflow_rescaling_long_alignment_many_tips(P, orc):
 
 
 # ------------------------------------------------------------------ GMH step (lock-step, P20)
-def _lockstep(P, orc, wl, N, steps, seed, K=None, precision=64):
+def _lockstep(P, orc, wl, N, steps, seed, K=None, precision=64, incremental=False):
     codes = wl["codes"]
     pi = orc.base_freqs(codes)
     u = orc.default_rate(pi)
     theta0 = wl["theta0"]
     parent, age = orc.upgma(codes, theta0)
     gl = orc.log_likelihood(codes, parent, age, pi, u)
-    ctx = _ctx(P, codes, theta0, tree=(parent, age), precision=precision, max_proposals=N, max_samples=16)
+    ctx = _ctx(P, codes, theta0, tree=(parent, age), precision=precision, max_proposals=N, max_samples=16,
+               incremental=incremental)
     K = N if K is None else K
     height = age.max()
     skipped = 0
@@ -142,6 +143,37 @@ def test_lockstep_c2_shape(P, orc):
 def test_lockstep_n24_ragged(P, orc):
     wl = synth.workload("c3", L=257, N=48)
     assert _lockstep(P, orc, wl, 48, 6, 77) <= 1
+
+
+@pytest.mark.parametrize("name,over,N,steps", [("c1", {}, 16, 30), ("c2", {"L": 300}, 64, 10),
+                                               ("c3", {"L": 257, "N": 48}, 48, 6), ("c4", {"n": 128, "L": 300}, 32, 4)])
+def test_lockstep_incremental_rescoring(P, orc, name, over, N, steps):
+    """incremental rescoring gives the oracle's (full-pruning)
+    likelihoods to 1e-9 and the same draws."""
+    wl = synth.workload(name, **over)
+    assert _lockstep(P, orc, wl, N, steps, wl["chain_seed"], incremental=True) <= 1
+
+
+def test_incremental_chain_matches_full_pruning(P):
+    """Free-running: the incremental context keeps its stored partials in step
+    with the generator over many commits (same chain as full pruning)."""
+    wl = synth.workload("c2", L=400)
+    rows = synth.to_strings(wl["codes"])
+    tree = (wl["true_parent"], wl["true_age"])
+    out = []
+    for inc in (False, True):
+        c = P.Context(rows, wl["theta0"], init_tree=tree, max_proposals=64, max_samples=6400, burnin_steps=20,
+                      incremental=inc)
+        c.mpcgs_sample(64, 6400, 3)
+        out.append(c.mpcgs_get_samples())
+        _, _, gl, _ = c.mpcgs_get_state()
+        # the stored partials still describe the generator: rescoring it from scratch agrees
+        p, a, _, _ = c.mpcgs_get_state()
+        assert abs(c.mpcgs_score_trees(p[None], a[None])[0] - gl) <= 1e-9 * abs(gl)
+    full, inc = out
+    same = np.cumprod(full["slot"] == inc["slot"]).sum()
+    assert same >= 2000, same   # identical until a near-threshold draw (if any)
+    assert np.allclose(full["logL"][:same], inc["logL"][:same], rtol=1e-10, atol=0)
 
 
 def test_lockstep_fp32_loglik_only(P, orc):
