@@ -11,6 +11,8 @@
 // proposal and site falls from n-1 nodes to 2 + depth(A) nodes.  After each
 // draw k_commit_incr rewrites the changed nodes of the new generator.
 // Results equal full pruning up to FP rounding order.
+#include <type_traits>
+
 #include "arith.cuh"
 #include "common.cuh"
 #include "kernels.cuh"
@@ -18,7 +20,8 @@
 namespace mpcgs {
 
 constexpr int INCR_THREADS = 128;
-constexpr int INCR_PG = 8;  // proposals per CTA (per-thread accumulators)
+constexpr int INCR_PG = 8;   // proposals per CTA (per-thread accumulators)
+constexpr int INCR_Q = 4;    // proposals whose ancestor chains advance together
 
 // node c at `site`: tip -> indicator vector, exponent 0; interior -> GL, GE
 template <typename T>
@@ -107,26 +110,34 @@ __global__ void __launch_bounds__(256) k_commit_incr(DevState s) {
 
 // ---------------------------------------------------------------- proposal scores
 // Grid (site tiles, ceil(count / INCR_PG)); each CTA scores INCR_PG proposals of
-// this rank over one tile.  Per site the three children's partials are loaded
-// once and reused by every proposal of the CTA.
+// this rank over one tile.  Per site, the three children's partials and the
+// ancestors' sibling factors B_a = br(L_sib(a)) (proposal-independent) are
+// computed once -- B_a into shared memory -- and reused by every proposal:
+// a proposal then costs two node combines plus one branch and one product per
+// ancestor.
+constexpr int INCR_DC = 8;  // ancestor levels cached in shared memory per site
+
 template <typename T>
 __global__ void __launch_bounds__(INCR_THREADS) k_score_incr(DevState s, IncrArgs a) {
-    __shared__ int sh_path[128], sh_sib[128];
+    __shared__ int sh_sib[128];
     __shared__ double sh_pe[4 * 128];   // e, em of the path branches and of the siblings' branches
     __shared__ int sh_xyz[INCR_PG][4];
     __shared__ double sh_ee[INCR_PG][10];
     __shared__ double s_red[INCR_THREADS / 32];
     __shared__ bool s_last;
+    using T2 = typename std::conditional<sizeof(T) == 8, double2, float2>::type;
+    __shared__ __align__(16) T2 sB[INCR_DC][2][INCR_THREADS];  // B_a of this thread's current site (conflict-free halves)
+    __shared__ int sBE[INCR_DC][INCR_THREADS];
     const int tid = threadIdx.x, tile = blockIdx.x;
     const int p0 = blockIdx.y * INCR_PG;
     const int np = min(INCR_PG, a.count - p0);
     const int c0 = s.ctx_i[6], c1 = s.ctx_i[7], c2 = s.ctx_i[8];
     const bool rootcase = s.ctx_i[3] != 0;
-    const int d = s.ctx_i[11];
+    const int d = rootcase ? 0 : s.ctx_i[11];
     const int dc = min(d, 128);  // ancestors whose ids / factors are cached in shared memory
+    const int db = min(d, INCR_DC);
     for (int i = tid; i < dc; i += INCR_THREADS) {
         const int an = s.path[i], sb = s.pathsib[i];
-        sh_path[i] = an;
         sh_sib[i] = sb;
         sh_pe[4 * i + 0] = s.e[an];
         sh_pe[4 * i + 1] = s.em[an];
@@ -151,66 +162,99 @@ __global__ void __launch_bounds__(INCR_THREADS) k_score_incr(DevState s, IncrArg
         const int k0 = load_node<T>(s, c0, site, L0);
         const int k1 = load_node<T>(s, c1, site, L1);
         const int k2 = load_node<T>(s, c2, site, L2);
+        for (int i = 0; i < db; ++i) {  // B_a, proposal-independent: once per site
+            T v[4];
+            const int ks = load_node<T>(s, sh_sib[i], site, v);
+            branch<T>(v, (T)sh_pe[4 * i + 2], (T)sh_pe[4 * i + 3], pi);
+            T2 qa, qb;
+            qa.x = v[0]; qa.y = v[1]; qb.x = v[2]; qb.y = v[3];
+            sB[i][0][tid] = qa;
+            sB[i][1][tid] = qb;
+            sBE[i][tid] = ks;
+        }
+        // INCR_Q proposals advance together: independent chains give the FP pipe ILP
 #pragma unroll
-        for (int j = 0; j < INCR_PG; ++j) {
-            if (j >= np) break;
-            const int x = sh_xyz[j][0], y = sh_xyz[j][1];
-            const double* ee = sh_ee[j];
-            T vx[4], vy[4], vz[4];
-            int kx, ky, kz;
-            // pair code 0 = (c1,c2) | c3, 1 = (c1,c3) | c2, 2 = (c2,c3) | c1 (S14)
-            if (x == c0 && y == c1) {
+        for (int j0 = 0; j0 < INCR_PG; j0 += INCR_Q) {
+            if (j0 >= np) break;
+            T vx[INCR_Q][4];
+            int kc[INCR_Q];
 #pragma unroll
-                for (int i = 0; i < 4; ++i) { vx[i] = L0[i]; vy[i] = L1[i]; vz[i] = L2[i]; }
-                kx = k0; ky = k1; kz = k2;
-            } else if (x == c0) {
+            for (int q = 0; q < INCR_Q; ++q) {
+                const int j = min(j0 + q, np - 1);  // tail: recompute the last proposal, not stored
+                const int x = sh_xyz[j][0], y = sh_xyz[j][1];
+                const double* ee = sh_ee[j];
+                T vy[4], vz[4];
+                int kx, ky, kz;
+                // pair code 0 = (c1,c2) | c3, 1 = (c1,c3) | c2, 2 = (c2,c3) | c1 (S14)
+                if (x == c0 && y == c1) {
 #pragma unroll
-                for (int i = 0; i < 4; ++i) { vx[i] = L0[i]; vy[i] = L2[i]; vz[i] = L1[i]; }
-                kx = k0; ky = k2; kz = k1;
-            } else {
+                    for (int i = 0; i < 4; ++i) { vx[q][i] = L0[i]; vy[i] = L1[i]; vz[i] = L2[i]; }
+                    kx = k0; ky = k1; kz = k2;
+                } else if (x == c0) {
 #pragma unroll
-                for (int i = 0; i < 4; ++i) { vx[i] = L1[i]; vy[i] = L2[i]; vz[i] = L0[i]; }
-                kx = k1; ky = k2; kz = k0;
+                    for (int i = 0; i < 4; ++i) { vx[q][i] = L0[i]; vy[i] = L2[i]; vz[i] = L1[i]; }
+                    kx = k0; ky = k2; kz = k1;
+                } else {
+#pragma unroll
+                    for (int i = 0; i < 4; ++i) { vx[q][i] = L1[i]; vy[i] = L2[i]; vz[i] = L0[i]; }
+                    kx = k1; ky = k2; kz = k0;
+                }
+                kc[q] = combine<T>(vx[q], kx, (T)ee[0], (T)ee[1], vy, ky, (T)ee[2], (T)ee[3], pi);      // T
+                kc[q] = combine<T>(vx[q], kc[q], (T)ee[6], (T)ee[7], vz, kz, (T)ee[4], (T)ee[5], pi);   // Par
             }
-            int kc = combine<T>(vx, kx, (T)ee[0], (T)ee[1], vy, ky, (T)ee[2], (T)ee[3], pi);   // T
-            kc = combine<T>(vx, kc, (T)ee[6], (T)ee[7], vz, kz, (T)ee[4], (T)ee[5], pi);         // Par
-            if (!rootcase) {
-                T pe = (T)ee[8], pem = (T)ee[9];  // branch Par -> A
-                for (int i = 0; i < d; ++i) {
-                    int sb;
-                    T se, sem, ae, aem;
-                    if (i < dc) {
-                        sb = sh_sib[i];
-                        ae = (T)sh_pe[4 * i + 0]; aem = (T)sh_pe[4 * i + 1];
-                        se = (T)sh_pe[4 * i + 2]; sem = (T)sh_pe[4 * i + 3];
-                    } else {
-                        const int an = s.path[i];
-                        sb = s.pathsib[i];
-                        ae = (T)s.e[an]; aem = (T)s.em[an]; se = (T)s.e[sb]; sem = (T)s.em[sb];
+            for (int i = 0; i < d; ++i) {
+                T bs[4];
+                int ks;
+                if (i < db) {
+                    const T2 qa = sB[i][0][tid], qb = sB[i][1][tid];
+                    bs[0] = qa.x; bs[1] = qa.y; bs[2] = qb.x; bs[3] = qb.y;
+                    ks = sBE[i][tid];
+                } else {  // deep paths: recompute the sibling factor
+                    const int sb = i < dc ? sh_sib[i] : s.pathsib[i];
+                    ks = load_node<T>(s, sb, site, bs);
+                    branch<T>(bs, (T)s.e[sb], (T)s.em[sb], pi);
+                }
+#pragma unroll
+                for (int q = 0; q < INCR_Q; ++q) {
+                    const int j = min(j0 + q, np - 1);
+                    T pe, pem;  // branch from the previous path node: Par -> A, then a(i-1) -> a(i)
+                    if (i == 0) { pe = (T)sh_ee[j][8]; pem = (T)sh_ee[j][9]; }
+                    else if (i - 1 < dc) { pe = (T)sh_pe[4 * (i - 1) + 0]; pem = (T)sh_pe[4 * (i - 1) + 1]; }
+                    else { const int an = s.path[i - 1]; pe = (T)s.e[an]; pem = (T)s.em[an]; }
+                    branch<T>(vx[q], pe, pem, pi);
+#pragma unroll
+                    for (int r = 0; r < 4; ++r) vx[q][r] *= bs[r];
+                    const int kr = rescale_k(vx[q]);
+                    if (kr) {
+                        const T f = pow2(kr, T(0));
+                        vx[q][0] *= f; vx[q][1] *= f; vx[q][2] *= f; vx[q][3] *= f;
                     }
-                    T vs[4];
-                    const int ks = load_node<T>(s, sb, site, vs);
-                    kc = combine<T>(vx, kc, pe, pem, vs, ks, se, sem, pi);
-                    pe = ae;
-                    pem = aem;
+                    kc[q] += ks + kr;
                 }
             }
-            // Eq. 21 at the root, multiplied into this proposal's accumulator
-            T ls = pi[0] * vx[0];
-            ls = fma(pi[1], vx[1], ls);
-            ls = fma(pi[2], vx[2], ls);
-            ls = fma(pi[3], vx[3], ls);
-            mant[j] *= (double)ls;
-            const int hi = __double2hiint(mant[j]);
-            const int ex = ((hi >> 20) & 2047) - 1023;
-            if (ex > -1023) {
-                mant[j] = __hiloint2double((hi & 0x800FFFFF) | (1023 << 20), __double2loint(mant[j]));
-                expo[j] += ex;
+#pragma unroll
+            for (int q = 0; q < INCR_Q; ++q) {
+                const int j = j0 + q;
+                if (j >= np) break;
+                // Eq. 21 at the root, multiplied into this proposal's accumulator
+                T ls = pi[0] * vx[q][0];
+                ls = fma(pi[1], vx[q][1], ls);
+                ls = fma(pi[2], vx[q][2], ls);
+                ls = fma(pi[3], vx[q][3], ls);
+                mant[j] *= (double)ls;
+                const int hi = __double2hiint(mant[j]);
+                const int ex = ((hi >> 20) & 2047) - 1023;
+                if (ex > -1023) {
+                    mant[j] = __hiloint2double((hi & 0x800FFFFF) | (1023 << 20), __double2loint(mant[j]));
+                    expo[j] += ex;
+                }
+                expo[j] -= kc[q];
             }
-            expo[j] -= kc;
         }
     }
-    for (int j = 0; j < np; ++j) {
+#pragma unroll
+    for (int j = 0; j < INCR_PG; ++j) {
+        if (j >= np) break;
         double ll = (mant[j] > 0.0) ? log(mant[j]) + (double)expo[j] * 0.69314718055994530942 : -INFINITY;
 #pragma unroll
         for (int off = 16; off > 0; off >>= 1) ll += __shfl_down_sync(0xffffffffu, ll, off);
