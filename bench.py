@@ -169,8 +169,10 @@ def workload_config(args, wl):
             "n_seq": n, "n_sites": L, "proposals_per_step": wl["N"], "theta0": wl["theta0"],
             "precision": args.precision, "l2": "flushed (256 MiB write) between timed steps",
             "parallelism": f"proposal-sharded x{args.gpus}", "init_tree": "synthetic true tree (ms-style)",
-            "scoring": "incremental rescoring (f2): partials/s counts the full-pruning equivalent n-1 nodes "
-                       "per proposal and site" if getattr(args, "incremental", False) else "full pruning (5.2.2)"}
+            "scoring": ("incremental rescoring (f2): partials/s counts the full-pruning equivalent n-1 nodes "
+                        "per proposal and site" if getattr(args, "incremental", False) else "full pruning (5.2.2)")
+            + ("; compressed site patterns (f3): partials/s counts all L columns" if getattr(args, "compress", False)
+               else "")}
 
 
 def main():
@@ -187,6 +189,8 @@ def main():
     ap.add_argument("--cpu-seconds", type=float, default=12.0)
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--no-incremental-block", action="store_true")
+    ap.add_argument("--compress", action="store_true",
+                    help="score distinct alignment columns weighted by count (SURVEY 8(f) f3)")
     ap.add_argument("--incremental", action="store_true",
                     help="score proposals by incremental rescoring (SURVEY 8(f) f2) instead of full pruning")
     args = ap.parse_args()
@@ -243,7 +247,7 @@ def main():
 
     ctx = P.Context(rows, wl["theta0"], precision=args.precision, max_proposals=N, max_samples=N * total_steps,
                     init_tree=(wl["true_parent"], wl["true_age"]), rank=rank, world=world, nccl_id=nccl_id,
-                    stream=stream, incremental=args.incremental)
+                    stream=stream, incremental=args.incremental, compress_patterns=args.compress)
     # warm-up (untimed): W steps
     ctx.mpcgs_sample(N, N * args.warmup, wl["chain_seed"])
     ctx.mpcgs_set_timing(3)   # per-step + per-prune CUDA events, L2 flush between steps

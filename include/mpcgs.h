@@ -91,6 +91,8 @@ typedef struct {
                               1: incremental rescoring: the generator's partials
                               of all nodes and sites stay in device memory and a proposal
                               recomputes only T, Par and the ancestors of Par (L1390-1398) */
+    int32_t compress_patterns; /* 1: score each distinct alignment column once, weighted by its
+                              count (exact by site independence, L714-716) */
 } mpcgs_config;
 
 /* [host-only] Fill cfg with defaults: empirical pi, default u, precision 64, burn-in 0,
@@ -173,6 +175,8 @@ mpcgs_status mpcgs_step_finish(mpcgs_ctx* ctx, int64_t step, int32_t n_proposals
 mpcgs_status mpcgs_get_samples(mpcgs_ctx* ctx, int64_t first, int64_t count, double* S,
                                double* logL, int64_t* step, int32_t* slot);
 int64_t mpcgs_num_samples(const mpcgs_ctx* ctx);
+/* Sites the kernels score: distinct columns with compress_patterns, else n_sites. */
+int32_t mpcgs_num_patterns(const mpcgs_ctx* ctx);
 
 /* Re-drive: theta0 <- theta (L791-797).  Cached P(D|G) stays valid (Eq. 23). */
 mpcgs_status mpcgs_set_theta0(mpcgs_ctx* ctx, double theta0);

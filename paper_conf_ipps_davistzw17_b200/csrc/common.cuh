@@ -148,6 +148,7 @@ struct DevState {
     double u;       // F81 rate (S3)
     double theta0;  // driving value
     const uint8_t* codes;  // [n][Lpad], 0..3
+    const double* site_w;  // [L] pattern counts when sites are compressed patterns (f3), else nullptr
     // generator (chain state)
     int32_t *parent, *left, *right, *need;  // [nn] (left/right/need valid for interior)
     double *age, *e, *em;                   // [nn]; e/em of the branch above each node

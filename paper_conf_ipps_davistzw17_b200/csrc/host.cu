@@ -60,6 +60,7 @@ struct mpcgs_ctx {
     int n = 0, L = 0, nn = 0, Lpad = 0, nops = 0, depth = 0, precision = 64;
     int world = 1, rank = 0, burnin = 0;
     bool incremental = false;
+    int L_orig = 0;          // alignment columns (L = scored sites: patterns if compressed)
     int Nmax = 0;
     int64_t Mmax = 0;
     double theta0 = 0.0, sample_theta0 = 0.0;
@@ -112,7 +113,7 @@ mpcgs_status fail(mpcgs_ctx* c, mpcgs_status st, const std::string& msg) {
 struct Layout {
     size_t codes, codes2, parent, left, right, need, age, e, em, gen, ctx_i, ctx_d, tau, len, lcnt, entry, omega, fixed;
     size_t tree_need, rec, sched_op, sched_e, tile_part, tile_cnt, sS, sL, sStep, sSlot, counters, last_draws, theta_buf,
-        theta_cnt, score_out, GL, GE, path, pathsib, cpath, csib, ixyz, iee, cinfo, gen_order, total;
+        theta_cnt, score_out, site_w, GL, GE, path, pathsib, cpath, csib, ixyz, iee, cinfo, gen_order, total;
     int tiles_max;
 };
 
@@ -166,6 +167,7 @@ Layout layout(int n, int L, int Nmax, int64_t Mmax, int precision, int increment
     y.theta_buf = take(8 * (size_t)(2 * MPCGS_MAX_GRID + 3 * 296 + 16));
     y.theta_cnt = take(16);
     y.score_out = take(8 * (size_t)Nmax);
+    y.site_w = take(8 * (size_t)L);
     const size_t tsz = precision == 32 ? 4 : 8;
     y.GL = take(incremental ? 4 * tsz * (size_t)(n - 1) * Lpad : 0);
     y.GE = take(incremental ? 4 * (size_t)(n - 1) * Lpad : 0);
@@ -351,6 +353,7 @@ PruneArgs prune_args(mpcgs_ctx* c, int ntrees_global, double* out, int out_first
     PruneArgs a{};
     a.codes = c->s.codes;
     a.codes2 = c->codes2;
+    a.site_w = c->s.site_w;
     a.W2 = codes2_words(c->L);
     a.Lpad = c->Lpad;
     a.L = c->L;
@@ -642,7 +645,8 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
     if (!out) return MPCGS_E_ARG;
     *out = nullptr;
     if (!aln || !cfg || !aln->rows) return MPCGS_E_ARG;
-    const int n = aln->n_seq, L = aln->n_sites;
+    const int n = aln->n_seq;
+    int L = aln->n_sites;  // becomes the number of scored sites (patterns) under compression
     if (n < 3 || n > MPCGS_MAX_SEQ || L < 1 || !(theta0 > 0.0) || !std::isfinite(theta0)) return MPCGS_E_ARG;
     if (cfg->precision != 32 && cfg->precision != 64) return MPCGS_E_ARG;
     if (cfg->max_proposals < 1 || cfg->max_proposals > MPCGS_MAX_PROPOSALS || cfg->max_samples < 0) return MPCGS_E_ARG;
@@ -697,8 +701,41 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
         upgma(n, L, codes.data(), theta0, parent.data(), age.data());
     }
     // device memory
+    // site-pattern compression (f3): distinct columns in lexicographic order + counts
+    c->L_orig = L;
+    std::vector<double> weights;
+    int Ls = L;
+    if (cfg->compress_patterns) {
+        std::vector<int> idx(L);
+        for (int s2 = 0; s2 < L; ++s2) idx[s2] = s2;
+        auto colcmp = [&](int a2, int b2) {
+            for (int i = 0; i < n; ++i) {
+                const uint8_t x = codes[(size_t)i * L + a2], y2 = codes[(size_t)i * L + b2];
+                if (x != y2) return x < y2;
+            }
+            return false;
+        };
+        std::stable_sort(idx.begin(), idx.end(), colcmp);
+        std::vector<int> reps;
+        for (int k = 0; k < L; ++k) {
+            if (k == 0 || colcmp(idx[k - 1], idx[k])) {
+                reps.push_back(idx[k]);
+                weights.push_back(1.0);
+            } else {
+                weights.back() += 1.0;
+            }
+        }
+        Ls = (int)reps.size();
+        std::vector<uint8_t> comp((size_t)n * Ls);
+        for (int i = 0; i < n; ++i)
+            for (int k = 0; k < Ls; ++k) comp[(size_t)i * Ls + k] = codes[(size_t)i * L + reps[k]];
+        codes.swap(comp);
+    }
+    L = Ls;
+    c->L = L;
+    c->Lpad = (L + 15) & ~15;
     c->incremental = cfg->incremental != 0;
-    Layout y = layout(n, L, c->Nmax, c->Mmax, c->precision, c->incremental);
+    Layout y = layout(n, Ls, c->Nmax, c->Mmax, c->precision, c->incremental);
     mpcgs_status st = MPCGS_OK;
     do {
         if (cudaStreamCreateWithFlags(&c->work, cudaStreamNonBlocking) != cudaSuccess ||
@@ -776,6 +813,7 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
         c->theta_cnt = (unsigned*)(b + y.theta_cnt);
         c->score_out = (double*)(b + y.score_out);
         c->codes2 = (uint32_t*)(b + y.codes2);
+        s.site_w = cfg->compress_patterns ? (const double*)(b + y.site_w) : nullptr;
         if ((st = enter(c))) break;
         if (cudaMemsetAsync(c->ws, 0, y.total, c->work) != cudaSuccess) { st = fail(c, MPCGS_E_CUDA, "memset"); break; }
         std::vector<uint8_t> padded((size_t)n * c->Lpad, 0);
@@ -788,6 +826,11 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
         if (cudaMemcpyAsync((void*)s.codes, padded.data(), padded.size(), cudaMemcpyHostToDevice, c->work) != cudaSuccess ||
             cudaMemcpyAsync(c->codes2, packed.data(), packed.size() * 4, cudaMemcpyHostToDevice, c->work) != cudaSuccess) {
             st = fail(c, MPCGS_E_CUDA, "codes upload");
+            break;
+        }
+        if (s.site_w &&
+            cudaMemcpyAsync((void*)s.site_w, weights.data(), 8 * weights.size(), cudaMemcpyHostToDevice, c->work) != cudaSuccess) {
+            st = fail(c, MPCGS_E_CUDA, "pattern weights upload");
             break;
         }
         if ((st = upload_state(c, parent.data(), age.data()))) break;
@@ -954,6 +997,8 @@ mpcgs_status mpcgs_last_timing(const mpcgs_ctx* c, double* loop_ms, double* prun
 }
 
 int64_t mpcgs_num_samples(const mpcgs_ctx* c) { return c ? c->nsamples : 0; }
+
+int32_t mpcgs_num_patterns(const mpcgs_ctx* c) { return c ? c->L : 0; }
 
 mpcgs_status mpcgs_get_samples(mpcgs_ctx* c, int64_t first, int64_t count, double* S, double* logL, int64_t* step,
                                int32_t* slot) {

@@ -150,13 +150,7 @@ __global__ void __launch_bounds__(INCR_THREADS) k_score_incr(DevState s, IncrArg
     const T pi[4] = {(T)s.pi[0], (T)s.pi[1], (T)s.pi[2], (T)s.pi[3]};
     const int s_begin = tile * a.sites_per_cta;
     const int s_end = min(s.L, s_begin + a.sites_per_cta);
-    double mant[INCR_PG];
-    int expo[INCR_PG];
-#pragma unroll
-    for (int j = 0; j < INCR_PG; ++j) {
-        mant[j] = 1.0;
-        expo[j] = 0;
-    }
+    SiteAcc acc[INCR_PG];
     for (int site = s_begin + tid; site < s_end; site += INCR_THREADS) {
         T L0[4], L1[4], L2[4];
         const int k0 = load_node<T>(s, c0, site, L0);
@@ -241,21 +235,14 @@ __global__ void __launch_bounds__(INCR_THREADS) k_score_incr(DevState s, IncrArg
                 ls = fma(pi[1], vx[q][1], ls);
                 ls = fma(pi[2], vx[q][2], ls);
                 ls = fma(pi[3], vx[q][3], ls);
-                mant[j] *= (double)ls;
-                const int hi = __double2hiint(mant[j]);
-                const int ex = ((hi >> 20) & 2047) - 1023;
-                if (ex > -1023) {
-                    mant[j] = __hiloint2double((hi & 0x800FFFFF) | (1023 << 20), __double2loint(mant[j]));
-                    expo[j] += ex;
-                }
-                expo[j] -= kc[q];
+                acc[j].add((double)ls, kc[q], s.site_w, site);
             }
         }
     }
 #pragma unroll
     for (int j = 0; j < INCR_PG; ++j) {
         if (j >= np) break;
-        double ll = (mant[j] > 0.0) ? log(mant[j]) + (double)expo[j] * 0.69314718055994530942 : -INFINITY;
+        double ll = acc[j].total();
 #pragma unroll
         for (int off = 16; off > 0; off >>= 1) ll += __shfl_down_sync(0xffffffffu, ll, off);
         if ((tid & 31) == 0) s_red[tid >> 5] = ll;

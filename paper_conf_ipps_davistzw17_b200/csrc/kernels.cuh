@@ -29,6 +29,7 @@ struct PruneArgs {
     const uint32_t* sched_op;  // [ntrees][nops]
     const void* sched_e;       // [ntrees][nops] float4 / double4
     int tiles, sites_per_cta;
+    const double* site_w;      // [L] pattern counts (compressed sites, f3) or nullptr
     const int32_t* tree_need;  // [ntrees] register need of each tree's schedule (nullable)
     int need_cap;              // set by launch_prune: largest need the table kernel serves
     double* tile_part;         // [ntrees][tiles]

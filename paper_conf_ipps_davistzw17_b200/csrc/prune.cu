@@ -97,8 +97,7 @@ __global__ void __launch_bounds__(PRUNE_THREADS) k_prune(PruneArgs a) {
     const int s_begin = tile * a.sites_per_cta;
     const int s_end = min(a.L, s_begin + a.sites_per_cta);
 
-    double mant = 1.0;  // product of site likelihoods = mant * 2^expo
-    int expo = 0;
+    SiteAcc acc;
     T R[D][4];
 #pragma unroll
     for (int i = 0; i < D; ++i)
@@ -122,17 +121,10 @@ __global__ void __launch_bounds__(PRUNE_THREADS) k_prune(PruneArgs a) {
         ls = fma(pi[1], R[0][1], ls);
         ls = fma(pi[2], R[0][2], ls);
         ls = fma(pi[3], R[0][3], ls);
-        mant *= (double)ls;
-        int hi = __double2hiint(mant);
-        int ex = ((hi >> 20) & 2047) - 1023;
-        if (ex > -1023) {  // normal: move the exponent into expo, mantissa to [1, 2)
-            mant = __hiloint2double((hi & 0x800FFFFF) | (1023 << 20), __double2loint(mant));
-            expo += ex;
-        }
-        expo -= scale;
+        acc.add((double)ls, scale, a.site_w, site);
     }
     // ln of this thread's product; -inf if any site likelihood was 0 (S6)
-    double ll = (mant > 0.0) ? log(mant) + (double)expo * 0.69314718055994530942 : -INFINITY;
+    double ll = acc.total();
     if (s_begin + (int)threadIdx.x >= s_end) ll = 0.0;
 
     // block reduction in a fixed order
@@ -371,7 +363,10 @@ __host__ __device__ size_t tab_smem_bytes(int nops, int need) {
 }
 
 template <typename T, int DR, int SI, bool PT, int DMX>
-__global__ void __launch_bounds__(PRUNE_THREADS) k_prune_tab(PruneArgs a) {
+#ifndef MPCGS_MINB
+#define MPCGS_MINB 1
+#endif
+__global__ void __launch_bounds__(PRUNE_THREADS, MPCGS_MINB) k_prune_tab(PruneArgs a) {
     using E4 = typename Traits<T>::E4;
     using CD = Codes<SI>;
     constexpr uint32_t TABE = PT ? 32u : 16u;  // table entries per tip
@@ -471,8 +466,7 @@ __global__ void __launch_bounds__(PRUNE_THREADS) k_prune_tab(PruneArgs a) {
         if (small) s_op[op].y |= TAB_CHECK;
     }
 
-    double mant = 1.0;
-    int expo = 0;
+    SiteAcc acc;
     Stack<T, DR, SI> st;
     st.sm = s_spill + tid;
 #pragma unroll
@@ -511,20 +505,11 @@ __global__ void __launch_bounds__(PRUNE_THREADS) k_prune_tab(PruneArgs a) {
             ls = fma(pi[1], root[1], ls);
             ls = fma(pi[2], root[2], ls);
             ls = fma(pi[3], root[3], ls);
-            if (site0 + k < s_end) {  // sites past L (padding) are computed, not counted
-                mant *= (double)ls;
-                const int hi = __double2hiint(mant);
-                const int ex = ((hi >> 20) & 2047) - 1023;
-                if (ex > -1023) {
-                    mant = __hiloint2double((hi & 0x800FFFFF) | (1023 << 20), __double2loint(mant));
-                    expo += ex;
-                }
-                expo -= scale[k];
-            }
+            if (site0 + k < s_end) acc.add((double)ls, scale[k], a.site_w, site0 + k);  // padding not counted
         }
         __syncthreads();  // the buffer of batch b is refilled in iteration b+1
     }
-    double ll = (mant > 0.0) ? log(mant) + (double)expo * 0.69314718055994530942 : -INFINITY;
+    double ll = acc.total();
 
 #pragma unroll
     for (int off = 16; off > 0; off >>= 1) ll += __shfl_down_sync(0xffffffffu, ll, off);

@@ -39,6 +39,7 @@ class mpcgs_config(ctypes.Structure):
         ("init_age", ctypes.c_void_p), ("rank", ctypes.c_int32), ("world", ctypes.c_int32),
         ("nccl_id", ctypes.c_void_p), ("stream", ctypes.c_void_p), ("workspace", ctypes.c_void_p),
         ("workspace_bytes", ctypes.c_size_t), ("incremental", ctypes.c_int32),
+        ("compress_patterns", ctypes.c_int32),
     ]
 
 
@@ -66,6 +67,7 @@ _SIGS = {
     "mpcgs_step_finish": (_i32, [_P, _i64, _i32, _i32, _u64, _P]),
     "mpcgs_get_samples": (_i32, [_P, _i64, _i64, _P, _P, _P, _P]),
     "mpcgs_num_samples": (_i64, [_P]),
+    "mpcgs_num_patterns": (_i32, [_P]),
     "mpcgs_set_theta0": (_i32, [_P, _f64]),
     "mpcgs_em": (_i32, [_P, _i32, _i32, _i64, _u64, _i32, _P]),
     "mpcgs_get_model": (_i32, [_P, _P, _P]),
@@ -196,7 +198,8 @@ class Context:
 
     def __init__(self, rows, theta0, *, precision=64, burnin_steps=0, max_proposals=1024,
                  max_samples=1 << 20, base_freq=None, mu=0.0, init_tree=None, rank=0, world=1,
-                 nccl_id=None, stream=None, workspace=None, phylip=None, incremental=False):
+                 nccl_id=None, stream=None, workspace=None, phylip=None, incremental=False,
+                 compress_patterns=False):
         L = lib()
         cfg = mpcgs_config()
         L.mpcgs_config_default(ctypes.byref(cfg))
@@ -209,6 +212,7 @@ class Context:
         cfg.max_proposals = int(max_proposals)
         cfg.max_samples = int(max_samples)
         cfg.incremental = int(bool(incremental))
+        cfg.compress_patterns = int(bool(compress_patterns))
         self._keep = []
         if init_tree is not None:
             p = _i32a(init_tree[0])
@@ -322,6 +326,9 @@ class Context:
         self._chk(lib().mpcgs_step_finish(self.h, step, n_proposals, n_draws, seed, _ptr(draws)),
                   "step_finish")
         return draws
+
+    def mpcgs_num_patterns(self):
+        return int(lib().mpcgs_num_patterns(self.h))
 
     def mpcgs_num_samples(self):
         return int(lib().mpcgs_num_samples(self.h))

@@ -95,7 +95,7 @@ def test_underflow_rescaling_long_alignment_many_tips(P, orc):
 
 
 # ------------------------------------------------------------------ GMH step (lock-step, P20)
-def _lockstep(P, orc, wl, N, steps, seed, K=None, precision=64, incremental=False):
+def _lockstep(P, orc, wl, N, steps, seed, K=None, precision=64, incremental=False, compress=False):
     codes = wl["codes"]
     pi = orc.base_freqs(codes)
     u = orc.default_rate(pi)
@@ -103,7 +103,7 @@ def _lockstep(P, orc, wl, N, steps, seed, K=None, precision=64, incremental=Fals
     parent, age = orc.upgma(codes, theta0)
     gl = orc.log_likelihood(codes, parent, age, pi, u)
     ctx = _ctx(P, codes, theta0, tree=(parent, age), precision=precision, max_proposals=N, max_samples=16,
-               incremental=incremental)
+               incremental=incremental, compress_patterns=compress)
     K = N if K is None else K
     height = age.max()
     skipped = 0
@@ -152,6 +152,18 @@ def test_lockstep_incremental_rescoring(P, orc, name, over, N, steps):
     likelihoods to 1e-9 and the same draws."""
     wl = synth.workload(name, **over)
     assert _lockstep(P, orc, wl, N, steps, wl["chain_seed"], incremental=True) <= 1
+
+
+@pytest.mark.parametrize("incremental", [False, True])
+@pytest.mark.parametrize("theta_true", [1.0, 0.01])
+def test_lockstep_pattern_compression(P, orc, incremental, theta_true):
+    """scoring distinct columns weighted by their counts gives
+    the uncompressed oracle likelihoods (site independence, L714-716)."""
+    wl = synth.workload("c2", L=600, theta_true=theta_true)
+    ctx = _ctx(P, wl["codes"], wl["theta0"], compress_patterns=True, max_proposals=64, max_samples=16)
+    n_pat = ctx.mpcgs_num_patterns()
+    assert n_pat == np.unique(wl["codes"].T, axis=0).shape[0] < 600
+    assert _lockstep(P, orc, wl, 64, 6, wl["chain_seed"], incremental=incremental, compress=True) <= 1
 
 
 def test_incremental_chain_matches_full_pruning(P):
