@@ -123,26 +123,27 @@ __device__ __forceinline__ bool small4(const float (&r)[4]) {
 // a product kept as mantissa * 2^expo (one log at the end), or -- when the
 // sites are compressed patterns -- a sum of count * ln L_s.
 // `scale` is the power-of-two exponent removed from the site's vectors.
+template <bool W>  // W: compressed sites with weights (separate instantiation: keeps the log out of the hot loop)
 struct SiteAcc {
     double mant = 1.0, wlog = 0.0;
     int expo = 0;
     __device__ __forceinline__ void add(double ls, int scale, const double* __restrict__ w, int site) {
-        if (w) {
+        if constexpr (W) {
             wlog += w[site] * (log(ls) - (double)scale * 0.69314718055994530942);
-            return;
+        } else {
+            mant *= ls;
+            const int hi = __double2hiint(mant);
+            const int ex = ((hi >> 20) & 2047) - 1023;
+            if (ex > -1023) {  // normal: move the exponent into expo, mantissa to [1, 2)
+                mant = __hiloint2double((hi & 0x800FFFFF) | (1023 << 20), __double2loint(mant));
+                expo += ex;
+            }
+            expo -= scale;
         }
-        mant *= ls;
-        const int hi = __double2hiint(mant);
-        const int ex = ((hi >> 20) & 2047) - 1023;
-        if (ex > -1023) {  // normal: move the exponent into expo, mantissa to [1, 2)
-            mant = __hiloint2double((hi & 0x800FFFFF) | (1023 << 20), __double2loint(mant));
-            expo += ex;
-        }
-        expo -= scale;
     }
     __device__ __forceinline__ double total() const {
-        const double p = mant > 0.0 ? log(mant) + (double)expo * 0.69314718055994530942 : -INFINITY;
-        return p + wlog;
+        if constexpr (W) return wlog;
+        return mant > 0.0 ? log(mant) + (double)expo * 0.69314718055994530942 : -INFINITY;
     }
 };
 

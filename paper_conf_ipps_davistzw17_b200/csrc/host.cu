@@ -340,8 +340,8 @@ void upgma(int n, int L, const uint8_t* codes, double theta0, int32_t* parent, d
 // Sites per CTA: a multiple of the kernel's site batch, as many batches as keep
 // >= ~8 CTAs per SM busy.  Depends only on L and the GLOBAL tree count, so every
 // rank tiles (and sums) a proposal's sites identically (world-size invariance).
-void prune_tiling(int L, int ntrees_global, int precision, int& tiles, int& sites_per_cta) {
-    const int batch = prune_batch_sites(precision);
+void prune_tiling(int n, int L, int ntrees_global, int precision, int& tiles, int& sites_per_cta) {
+    const int batch = prune_batch_sites(n, precision);
     const long batches = (L + batch - 1) / batch;
     const long want = (long)148 * 8;
     const int per = (int)std::max<long>(1, std::min<long>(8, (ntrees_global * batches) / want));
@@ -361,7 +361,7 @@ PruneArgs prune_args(mpcgs_ctx* c, int ntrees_global, double* out, int out_first
     for (int i = 0; i < 4; ++i) a.pi[i] = c->s.pi[i];
     a.sched_op = c->s.sched_op;
     a.sched_e = c->s.sched_e;
-    prune_tiling(c->L, ntrees_global, c->precision, a.tiles, a.sites_per_cta);
+    prune_tiling(c->n, c->L, ntrees_global, c->precision, a.tiles, a.sites_per_cta);
     a.tree_need = c->s.tree_need;
     a.tile_part = c->s.tile_part;
     a.tile_cnt = c->s.tile_cnt;

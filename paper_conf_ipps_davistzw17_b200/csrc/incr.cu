@@ -117,7 +117,7 @@ __global__ void __launch_bounds__(256) k_commit_incr(DevState s) {
 // ancestor.
 constexpr int INCR_DC = 8;  // ancestor levels cached in shared memory per site
 
-template <typename T>
+template <typename T, bool W>
 __global__ void __launch_bounds__(INCR_THREADS) k_score_incr(DevState s, IncrArgs a) {
     __shared__ int sh_sib[128];
     __shared__ double sh_pe[4 * 128];   // e, em of the path branches and of the siblings' branches
@@ -150,7 +150,7 @@ __global__ void __launch_bounds__(INCR_THREADS) k_score_incr(DevState s, IncrArg
     const T pi[4] = {(T)s.pi[0], (T)s.pi[1], (T)s.pi[2], (T)s.pi[3]};
     const int s_begin = tile * a.sites_per_cta;
     const int s_end = min(s.L, s_begin + a.sites_per_cta);
-    SiteAcc acc[INCR_PG];
+    SiteAcc<W> acc[INCR_PG];
     for (int site = s_begin + tid; site < s_end; site += INCR_THREADS) {
         T L0[4], L1[4], L2[4];
         const int k0 = load_node<T>(s, c0, site, L0);
@@ -287,8 +287,14 @@ cudaError_t launch_commit_incr(const DevState& s, cudaStream_t st) {
 cudaError_t launch_score_incr(const DevState& s, const IncrArgs& a, cudaStream_t st) {
     if (a.count <= 0) return cudaSuccess;
     dim3 grid(a.tiles, (a.count + INCR_PG - 1) / INCR_PG);
-    if (s.precision == 32) k_score_incr<float><<<grid, INCR_THREADS, 0, st>>>(s, a);
-    else k_score_incr<double><<<grid, INCR_THREADS, 0, st>>>(s, a);
+    const bool w = s.site_w != nullptr;
+    if (s.precision == 32) {
+        if (w) k_score_incr<float, true><<<grid, INCR_THREADS, 0, st>>>(s, a);
+        else k_score_incr<float, false><<<grid, INCR_THREADS, 0, st>>>(s, a);
+    } else {
+        if (w) k_score_incr<double, true><<<grid, INCR_THREADS, 0, st>>>(s, a);
+        else k_score_incr<double, false><<<grid, INCR_THREADS, 0, st>>>(s, a);
+    }
     return cudaGetLastError();
 }
 

@@ -71,7 +71,7 @@ __device__ __forceinline__ void op_ss(T (&R)[D][4], const typename Traits<T>::E4
     case (OP_TS | ((S) << 2)): op_ts<T, D, S>(R, code, ed, codes, Lpad, site, pi, scale); break; \
     case (OP_SS | ((S) << 2)): op_ss<T, D, S>(R, ed, pi, scale); break;
 
-template <typename T, int D>
+template <typename T, int D, bool W>
 __global__ void __launch_bounds__(PRUNE_THREADS) k_prune(PruneArgs a) {
     using E4 = typename Traits<T>::E4;
     extern __shared__ __align__(16) unsigned char smem_raw[];
@@ -97,7 +97,7 @@ __global__ void __launch_bounds__(PRUNE_THREADS) k_prune(PruneArgs a) {
     const int s_begin = tile * a.sites_per_cta;
     const int s_end = min(a.L, s_begin + a.sites_per_cta);
 
-    SiteAcc acc;
+    SiteAcc<W> acc;
     T R[D][4];
 #pragma unroll
     for (int i = 0; i < D; ++i)
@@ -362,11 +362,13 @@ __host__ __device__ size_t tab_smem_bytes(int nops, int need) {
            sizeof(T) * (size_t)spill * SI * 4 * PRUNE_THREADS;
 }
 
-template <typename T, int DR, int SI, bool PT, int DMX>
-#ifndef MPCGS_MINB
-#define MPCGS_MINB 1
+#ifdef MPCGS_MINB  // tuning builds only: min CTAs per SM (caps registers)
+#define MPCGS_TAB_BOUNDS __launch_bounds__(PRUNE_THREADS, MPCGS_MINB)
+#else
+#define MPCGS_TAB_BOUNDS __launch_bounds__(PRUNE_THREADS)
 #endif
-__global__ void __launch_bounds__(PRUNE_THREADS, MPCGS_MINB) k_prune_tab(PruneArgs a) {
+template <typename T, int DR, int SI, bool PT, int DMX, bool W>
+__global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
     using E4 = typename Traits<T>::E4;
     using CD = Codes<SI>;
     constexpr uint32_t TABE = PT ? 32u : 16u;  // table entries per tip
@@ -466,7 +468,7 @@ __global__ void __launch_bounds__(PRUNE_THREADS, MPCGS_MINB) k_prune_tab(PruneAr
         if (small) s_op[op].y |= TAB_CHECK;
     }
 
-    SiteAcc acc;
+    SiteAcc<W> acc;
     Stack<T, DR, SI> st;
     st.sm = s_spill + tid;
 #pragma unroll
@@ -534,11 +536,31 @@ __global__ void __launch_bounds__(PRUNE_THREADS, MPCGS_MINB) k_prune_tab(PruneAr
     }
 }
 
+template <typename T, int D, bool W>
+static cudaError_t launch_flat_w(const PruneArgs& a, int ntrees, cudaStream_t st) {
+    size_t smem = (size_t)a.nops * (sizeof(typename Traits<T>::E4) + sizeof(uint32_t));
+    auto kern = k_prune<T, D, W>;
+    static size_t attr_bytes = 48 * 1024;  // raised once, outside graph capture (first launch is at init)
+    if (smem > attr_bytes) {
+        cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+        if (e != cudaSuccess) return e;
+        attr_bytes = smem;
+    }
+    dim3 grid(a.tiles, ntrees);
+    kern<<<grid, PRUNE_THREADS, smem, st>>>(a);
+    return cudaGetLastError();
+}
+
 template <typename T, int D>
 static cudaError_t launch_flat(const PruneArgs& a, int ntrees, cudaStream_t st) {
-    size_t smem = (size_t)a.nops * (sizeof(typename Traits<T>::E4) + sizeof(uint32_t));
-    auto kern = k_prune<T, D>;
-    static size_t attr_bytes = 48 * 1024;  // raised once, outside graph capture (first launch is at init)
+    return a.site_w ? launch_flat_w<T, D, true>(a, ntrees, st) : launch_flat_w<T, D, false>(a, ntrees, st);
+}
+
+template <typename T, int DR, int SI, bool PT, int DMX, bool W>
+static cudaError_t launch_tab_w(const PruneArgs& a, int ntrees, cudaStream_t st) {
+    const size_t smem = tab_smem_bytes<T, DR, SI, PT>(a.nops, a.need_cap);
+    auto kern = k_prune_tab<T, DR, SI, PT, DMX, W>;
+    static size_t attr_bytes = 48 * 1024;
     if (smem > attr_bytes) {
         cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
         if (e != cudaSuccess) return e;
@@ -551,17 +573,8 @@ static cudaError_t launch_flat(const PruneArgs& a, int ntrees, cudaStream_t st) 
 
 template <typename T, int DR, int SI, bool PT, int DMX>
 static cudaError_t launch_tab(const PruneArgs& a, int ntrees, cudaStream_t st) {
-    const size_t smem = tab_smem_bytes<T, DR, SI, PT>(a.nops, a.need_cap);
-    auto kern = k_prune_tab<T, DR, SI, PT, DMX>;
-    static size_t attr_bytes = 48 * 1024;
-    if (smem > attr_bytes) {
-        cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-        if (e != cudaSuccess) return e;
-        attr_bytes = smem;
-    }
-    dim3 grid(a.tiles, ntrees);
-    kern<<<grid, PRUNE_THREADS, smem, st>>>(a);
-    return cudaGetLastError();
+    return a.site_w ? launch_tab_w<T, DR, SI, PT, DMX, true>(a, ntrees, st)
+                    : launch_tab_w<T, DR, SI, PT, DMX, false>(a, ntrees, st);
 }
 
 int prune_depth_for(int n) {
@@ -579,13 +592,21 @@ int prune_max_need(int n) {
     return d < 1 ? 1 : d;
 }
 
-int prune_batch_sites(int precision) { return PRUNE_THREADS * (precision == 32 ? PRUNE_SI32 : PRUNE_SI64); }
+static bool product_tables(int n);
+// sites interleaved per thread: 4 for n <= 128 (product tables), 2 for larger
+// trees, whose codes / tables / spill levels take more shared memory
+static int prune_si(int n, int precision) {
+    if (!product_tables(n)) return 2;
+    return precision == 32 ? PRUNE_SI32 : PRUNE_SI64;
+}
+int prune_batch_sites(int n, int precision) { return PRUNE_THREADS * prune_si(n, precision); }
 
 // register need the table kernel serves (DR registers + PRUNE_SPILL shared levels);
 // deeper trees (rare) are scored by the flat kernel in a second pass
 int prune_need_cap(int n) { return std::min(prune_max_need(n), PRUNE_DR + PRUNE_SPILL); }
 
 static bool product_tables(int n) { return n <= 128; }
+constexpr int PRUNE_SI_LARGE = 2;
 
 bool prune_uses_tables(int n, int precision) {
     const int cap = prune_need_cap(n);
@@ -593,10 +614,10 @@ bool prune_uses_tables(int n, int precision) {
     size_t bytes;
     if (precision == 32)
         bytes = pt ? tab_smem_bytes<float, PRUNE_DR, PRUNE_SI32, true>(n - 1, cap)
-                   : tab_smem_bytes<float, PRUNE_DR, PRUNE_SI32, false>(n - 1, cap);
+                   : tab_smem_bytes<float, PRUNE_DR, PRUNE_SI_LARGE, false>(n - 1, cap);
     else
         bytes = pt ? tab_smem_bytes<double, PRUNE_DR, PRUNE_SI64, true>(n - 1, cap)
-                   : tab_smem_bytes<double, PRUNE_DR, PRUNE_SI64, false>(n - 1, cap);
+                   : tab_smem_bytes<double, PRUNE_DR, PRUNE_SI_LARGE, false>(n - 1, cap);
     return bytes <= 160 * 1024;
 }
 
@@ -632,7 +653,7 @@ static cudaError_t launch_typed(PruneArgs a, int ntrees, int depth, cudaStream_t
     const bool deep = prune_max_need(n) > a.need_cap && a.tree_need != nullptr;
     if (!deep) a.tree_need = nullptr;
     cudaError_t e = product_tables(n) ? launch_tab_dmx<T, SI, true>(a, ntrees, st)
-                                      : launch_tab_dmx<T, SI, false>(a, ntrees, st);
+                                      : launch_tab_dmx<T, PRUNE_SI_LARGE, false>(a, ntrees, st);
     if (e != cudaSuccess || !deep) return e;
     nl = 2;
     return launch_flat_depth<T>(a, ntrees, depth, st);  // trees with need > cap only

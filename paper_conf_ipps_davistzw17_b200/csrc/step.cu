@@ -13,11 +13,22 @@
 //                           CDF draws (L1140-1144), sample store, generator commit
 #include <algorithm>
 #include <cfloat>
+#include <cstdio>
 
 #include "common.cuh"
 #include "kernels.cuh"
 
 namespace mpcgs {
+
+#ifdef MPCGS_TIMESTAMPS
+__device__ long long g_ts[16];
+#define MPCGS_TS(i) do { if (threadIdx.x == 0 && blockIdx.x == 0) g_ts[i] = clock64(); } while (0)
+__device__ long long g_tp[8];
+#define MPCGS_TP(i) do { if (threadIdx.x == 0 && blockIdx.x == 0) g_tp[i] = clock64(); } while (0)
+#else
+#define MPCGS_TS(i) do { } while (0)
+#define MPCGS_TP(i) do { } while (0)
+#endif
 
 constexpr int CTX_THREADS = 256;
 constexpr int DRAW_THREADS = 1024;
@@ -102,6 +113,7 @@ __device__ int block_exclusive_scan(int v, int* s_warp, int* tot) {
 // device loop, at the end of k_draw (saves a launch per step).
 template <int NT>
 __device__ void context_body(const DevState& s, uint64_t seed, int64_t step_arg, double* csm) {
+    MPCGS_TS(5);
     const int n = s.n, nn = s.nn, nint = n - 1;
     double* sAge = csm;               // [n-1] ages of interior nodes (index v - n)
     double* sF = sAge + nint;         // [n] sorted fixed ages
@@ -145,6 +157,7 @@ __device__ void context_body(const DevState& s, uint64_t seed, int64_t step_arg,
         shd[3] = A < 0 ? CUDART_INF : s.age[A];
     }
     __syncthreads();
+    MPCGS_TS(6);
     const int T = sh[0], Par = sh[1];
     const double a1 = shd[1], a2 = shd[2], tA = shd[3];
     const bool rootcase = sh[3] != 0;
@@ -163,6 +176,7 @@ __device__ void context_body(const DevState& s, uint64_t seed, int64_t step_arg,
         sF[r] = av;
     }
     __syncthreads();
+    MPCGS_TS(7);
     if (tid == 0) {
         const int lo = upper_count(sF, nfixed, a1);  // fixed ages <= a(2): not cuts
         const int hi = lower_count(sF, nfixed, tA);  // fixed ages <  t_A
@@ -199,28 +213,31 @@ __device__ void context_body(const DevState& s, uint64_t seed, int64_t step_arg,
         sTau[m] = tA;
     }
     __syncthreads();
-    // per-interval bookkeeping and closed-form weights
-    for (int p = tid; p < m; p += NT) {
+    MPCGS_TS(8);
+    // per-interval bookkeeping and closed-form weights: one thread per (interval,
+    // weight), 6 weights per interval (the transcendentals dominate)
+    for (int q = tid; q < 6 * m; q += NT) {
+        const int p = q / 6, w = q - 6 * p;
         const double tp = sTau[p];
         const bool inf = rootcase && p == m - 1;
         const double len = inf ? CUDART_INF : sTau[p + 1] - tp;
         const int fixed_below = upper_count(sF, nfixed, tp);
         const int kids_below = (shd[0] <= tp) + (a1 <= tp) + (a2 <= tp);
         const int l = n - fixed_below - kids_below;
-        s.tau[p] = tp;
-        s.len[p] = len;
-        s.lcnt[p] = l;
-        sEntry[p] = (p >= 1 && has3 && tp == a2) ? 1 : 0;
-        const double th = s.theta0;
-        sW[p * 6 + 0] = what(1, 1, len, l, th, inf);
-        sW[p * 6 + 1] = what(2, 2, len, l, th, inf);
-        sW[p * 6 + 2] = what(2, 1, len, l, th, inf);
-        sW[p * 6 + 3] = what(3, 3, len, l, th, inf);
-        sW[p * 6 + 4] = what(3, 2, len, l, th, inf);
-        sW[p * 6 + 5] = what(3, 1, len, l, th, inf);
+        if (w == 0) {
+            s.tau[p] = tp;
+            s.len[p] = len;
+            s.lcnt[p] = l;
+            sEntry[p] = (p >= 1 && has3 && tp == a2) ? 1 : 0;
+        }
+        // rows (1,1) (2,2) (2,1) (3,3) (3,2) (3,1)
+        const int k = w == 0 ? 1 : (w < 3 ? 2 : 3);
+        const int kk = w == 0 ? 1 : (w == 1 ? 2 : (w == 2 ? 1 : (w == 3 ? 3 : (w == 4 ? 2 : 1))));
+        sW[p * 6 + w] = what(k, kk, len, l, s.theta0, inf);
     }
     if (tid == 0) sEntry[m] = 0;
     __syncthreads();
+    MPCGS_TS(9);
     // backward messages (L1005-1020): exactly one lineage at the ancestor
     if (tid == 0) {
         double b1 = 1.0, b2 = 0.0, b3 = 0.0;
@@ -243,6 +260,7 @@ __device__ void context_body(const DevState& s, uint64_t seed, int64_t step_arg,
         }
     }
     __syncthreads();
+    MPCGS_TS(10);
     // forward choice weights omega_p(k -> k') = W^_p(k -> k') beta_{p+1}(k' + entry_{p+1})
     for (int p = tid; p < m; p += NT) {
         const int en = sEntry[p + 1];
@@ -355,6 +373,12 @@ struct Walk {
 // Forward walk over the feasible intervals, young -> old (L1028-1034); RNG order
 // per interval: choice, event times, then the pair if the first coalescence
 // happens with three active lineages.
+// int words of k_propose's shared arrays (sL, sR, sNeed, sStack, sLc, sEn, sPar), rounded to even
+__host__ __device__ inline int propose_int_words(int n) {
+    const int w = 2 * (n - 1) + (2 * n - 1) + 2 * n + (n + 1) + (n + 2) + (2 * n - 1);
+    return (w + 1) & ~1;
+}
+
 struct WalkCtx {  // the step's interval context, staged in shared memory
     const double *tau, *len, *omega;
     const int *lcnt, *entry;
@@ -444,21 +468,27 @@ template <typename E4, typename ET>
 __global__ void __launch_bounds__(32) k_propose(DevState s, uint64_t seed, int64_t step_arg, int slot_first) {
     extern __shared__ __align__(16) int psm[];
     const int n = s.n, nn = s.nn, nint = n - 1;
-    int* sL = psm;             // [n-1] children of interior nodes (index v - n)
-    int* sR = sL + nint;       // [n-1]
-    int* sNeed = sR + nint;    // [nn]
-    int* sStack = sNeed + nn;  // [2n]
-    int* sLc = sStack + 2 * n;  // [n+1] inactive counts
-    int* sEn = sLc + n + 1;     // [n+2] entry flags
-    double* sTau = reinterpret_cast<double*>(psm + ((4 * n + 2 + 4 * n) & ~1) + 4);  // [n+2]
+    // shared copies of the generator and the step context: every sequential
+    // lookup of lane 0 (walk, need path, DFS emission) is a shared-memory access
+    int* sL = psm;                 // [n-1] children of interior nodes (index v - n)
+    int* sR = sL + nint;           // [n-1]
+    int* sNeed = sR + nint;        // [nn]
+    int* sStack = sNeed + nn;      // [2n]
+    int* sLc = sStack + 2 * n;     // [n+1] inactive counts
+    int* sEn = sLc + n + 1;        // [n+2] entry flags
+    int* sPar = sEn + n + 2;       // [nn] parents
+    double* sTau = reinterpret_cast<double*>(psm + propose_int_words(n));  // [n+2]
     double* sLen = sTau + n + 2;   // [n+1]
     double* sOm = sLen + n + 1;    // [9(n+1)]
+    double* sE = sOm + 9 * (n + 1);  // [nn] branch factor above each node (patched for the proposal)
+    double* sEm = sE + nn;           // [nn]
     __shared__ double sh_d[8];  // t1, t2, e/em of changed branches
     __shared__ int sh_i[8];
     __shared__ double sU[PRE_U];  // first uniforms of this slot's Philox stream
     const int lane = threadIdx.x;
     const int slot = slot_first + blockIdx.x;  // global slot 1..N
     const int local = blockIdx.x;
+    MPCGS_TP(0);
     const int64_t step = step_of(s, step_arg);
 
     const int T = s.ctx_i[0], Par = s.ctx_i[1], A = s.ctx_i[2];
@@ -466,6 +496,7 @@ __global__ void __launch_bounds__(32) k_propose(DevState s, uint64_t seed, int64
     const int k0 = s.ctx_i[4], m = s.ctx_i[5];
     const int c0 = s.ctx_i[6], c1 = s.ctx_i[7], c2 = s.ctx_i[8];
     const int nfixed = s.ctx_i[9], root = s.ctx_i[10];
+    const double ac0 = s.ctx_d[0], ac1 = s.ctx_d[1], ac2 = s.ctx_d[2], tAn = s.ctx_d[3];  // children's / ancestor's ages
 
     // stage the interval context (L2 reads once, coalesced) for lane 0's sequential walk
     for (int i = lane; i <= m; i += 32) {
@@ -477,6 +508,17 @@ __global__ void __launch_bounds__(32) k_propose(DevState s, uint64_t seed, int64
         }
     }
     for (int i = lane; i < 9 * m; i += 32) sOm[i] = s.omega[i];
+    for (int i = lane; i < nint; i += 32) {
+        sL[i] = s.left[n + i];
+        sR[i] = s.right[n + i];
+    }
+    for (int i = lane; i < nn; i += 32) {
+        sNeed[i] = i < n ? 0 : s.need[i];
+        sPar[i] = s.parent[i];
+        sE[i] = s.e[i];
+        sEm[i] = s.em[i];
+    }
+    MPCGS_TP(1);
     {  // one Philox block per lane: uniforms 2*lane, 2*lane+1 of (slot, step, PROPOSE)
         const U4 b = philox(U4{(uint32_t)lane, (uint32_t)slot, (uint32_t)step, TAG_PROPOSE}, (uint32_t)seed,
                             (uint32_t)(seed >> 32));
@@ -487,6 +529,7 @@ __global__ void __launch_bounds__(32) k_propose(DevState s, uint64_t seed, int64
     if (lane == 0) {
         const WalkCtx wc{sTau, sLen, sOm, sLc, sEn, s.theta0};
         Walk w = forward_walk(wc, m, k0, rootcase, seed, (uint32_t)slot, (uint32_t)step, sU);
+        MPCGS_TP(2);
         int pair = w.pair;
         double t1 = w.t1, t2 = w.t2;
         if (!w.ok) {
@@ -498,14 +541,10 @@ __global__ void __launch_bounds__(32) k_propose(DevState s, uint64_t seed, int64
             t2 = s.age[Par];
         }
         sh_i[0] = pair;
+        MPCGS_TP(3);
         sh_d[0] = t1;
         sh_d[1] = t2;
     }
-    for (int i = lane; i < nint; i += 32) {
-        sL[i] = s.left[n + i];
-        sR[i] = s.right[n + i];
-    }
-    for (int i = lane; i < nn; i += 32) sNeed[i] = i < n ? 0 : s.need[i];
     __syncwarp();
     const int pair = sh_i[0];
     const double t1 = sh_d[0], t2 = sh_d[1];
@@ -514,6 +553,9 @@ __global__ void __launch_bounds__(32) k_propose(DevState s, uint64_t seed, int64
     const int y = pair == 0 ? c1 : c2;
     const int z = pair == 0 ? c2 : (pair == 1 ? c1 : c0);
     const double u = s.u;
+    const double ax = x == c0 ? ac0 : (x == c1 ? ac1 : ac2);
+    const double ay = y == c0 ? ac0 : (y == c1 ? ac1 : ac2);
+    const double az = z == c0 ? ac0 : (z == c1 ? ac1 : ac2);
     if (lane == 0) {
         // younger new node keeps the target's id, older keeps the parent's (S15)
         sL[T - n] = min(x, y);
@@ -522,28 +564,29 @@ __global__ void __launch_bounds__(32) k_propose(DevState s, uint64_t seed, int64
         sR[Par - n] = max(T, z);
         sNeed[T] = su_need(sNeed[x], sNeed[y]);
         sNeed[Par] = su_need(sNeed[T], sNeed[z]);
-        for (int v = A; v >= 0; v = s.parent[v]) sNeed[v] = su_need(sNeed[sL[v - n]], sNeed[sR[v - n]]);
+        for (int v = A; v >= 0; v = sPar[v]) sNeed[v] = su_need(sNeed[sL[v - n]], sNeed[sR[v - n]]);
         s.tree_need[local] = sNeed[root];
     } else if (lane == 1) {
-        sh_d[2] = exp(-u * (t1 - s.age[x]));
-        sh_d[3] = -expm1(-u * (t1 - s.age[x]));
+        sh_d[2] = exp(-u * (t1 - ax));
+        sh_d[3] = -expm1(-u * (t1 - ax));
     } else if (lane == 2) {
-        sh_d[4] = exp(-u * (t1 - s.age[y]));
-        sh_d[5] = -expm1(-u * (t1 - s.age[y]));
+        sh_d[4] = exp(-u * (t1 - ay));
+        sh_d[5] = -expm1(-u * (t1 - ay));
     } else if (lane == 3) {
-        sh_d[6] = exp(-u * (t2 - s.age[z]));
-        sh_d[7] = -expm1(-u * (t2 - s.age[z]));
+        sh_d[6] = exp(-u * (t2 - az));
+        sh_d[7] = -expm1(-u * (t2 - az));
     }
     __shared__ double sh_e2[4];
     if (lane == 4) {
         sh_e2[0] = exp(-u * (t2 - t1));
         sh_e2[1] = -expm1(-u * (t2 - t1));
     } else if (lane == 5) {
-        const double lp = rootcase ? 0.0 : s.age[A] - t2;
+        const double lp = rootcase ? 0.0 : tAn - t2;
         sh_e2[2] = exp(-u * lp);
         sh_e2[3] = -expm1(-u * lp);
     }
     // S_G of the proposal: merge of the sorted fixed ages with {t1, t2} (Eq. 18 via
+    MPCGS_TP(4);
     // S = 2 sum_i (n - i) h_i over sorted coalescence ages)
     double base = 0.0, shift = 0.0;
     int cnt1 = 0, cnt2 = 0;
@@ -563,6 +606,7 @@ __global__ void __launch_bounds__(32) k_propose(DevState s, uint64_t seed, int64
     }
     __syncwarp();
     if (lane == 0) {
+    MPCGS_TP(5);
         const int r1 = 1 + cnt1, r2 = 2 + cnt2;
         const double S = 2.0 * (base - shift) + 2.0 * (double)(n - r1) * t1 + 2.0 * (double)(n - r2) * t2;
         double* rec = s.rec + (size_t)slot * REC;
@@ -570,17 +614,13 @@ __global__ void __launch_bounds__(32) k_propose(DevState s, uint64_t seed, int64
         rec[2] = t1;
         rec[3] = t2;
         rec[4] = (double)pair;
-        // post-order register schedule of the proposal tree
-        const double* ge = s.e;
-        const double* gem = s.em;
-        auto e_of = [&](int c, double& e, double& em) {
-            if (c == x) { e = sh_d[2]; em = sh_d[3]; }
-            else if (c == y) { e = sh_d[4]; em = sh_d[5]; }
-            else if (c == z) { e = sh_d[6]; em = sh_d[7]; }
-            else if (c == T) { e = sh_e2[0]; em = sh_e2[1]; }
-            else if (c == Par) { e = sh_e2[2]; em = sh_e2[3]; }
-            else { e = ge[c]; em = gem[c]; }
-        };
+        // post-order register schedule of the proposal tree; branch factors of the
+        // five changed branches patched into the shared copy
+        sE[x] = sh_d[2]; sEm[x] = sh_d[3];
+        sE[y] = sh_d[4]; sEm[y] = sh_d[5];
+        sE[z] = sh_d[6]; sEm[z] = sh_d[7];
+        sE[T] = sh_e2[0]; sEm[T] = sh_e2[1];
+        sE[Par] = sh_e2[2]; sEm[Par] = sh_e2[3];
         if (s.incremental) {
             int32_t* q = s.ixyz + 4 * (size_t)local;
             q[0] = x; q[1] = y; q[2] = z; q[3] = 0;
@@ -594,20 +634,24 @@ __global__ void __launch_bounds__(32) k_propose(DevState s, uint64_t seed, int64
             n, root, [&](int v) { return sL[v - n]; }, [&](int v) { return sR[v - n]; },
             [&](int v) { return sNeed[v]; },
             [&](int i, uint32_t code, int ca, int cb) {
-                double ea, ema, eb, emb;
-                e_of(ca, ea, ema);
-                e_of(cb, eb, emb);
                 op_out[i] = code;
                 E4 v;
-                v.x = (ET)ea; v.y = (ET)ema; v.z = (ET)eb; v.w = (ET)emb;
+                v.x = (ET)sE[ca]; v.y = (ET)sEm[ca]; v.z = (ET)sE[cb]; v.w = (ET)sEm[cb];
                 e_out[i] = v;
             },
             sStack);
+        MPCGS_TP(6);
+#ifdef MPCGS_TIMESTAMPS
+        if (blockIdx.x == 0 && step == 2)
+            printf("propose: stage %lld walk %lld patch %lld e+S %lld pre-dfs %lld dfs %lld\n", g_tp[1] - g_tp[0],
+                   g_tp[3] - g_tp[2], g_tp[4] - g_tp[3], g_tp[5] - g_tp[4], g_tp[2] - g_tp[1], g_tp[6] - g_tp[5]);
+#endif
     }
 }
 
 size_t propose_smem_bytes(int n) {
-    return sizeof(int) * ((size_t)((4 * n + 2 + 4 * n) & ~1) + 4) + sizeof(double) * ((size_t)(n + 2) + (n + 1) + 9 * (n + 1));
+    const size_t nn = 2 * (size_t)n - 1;
+    return sizeof(int) * (size_t)propose_int_words(n) + sizeof(double) * ((size_t)(n + 2) + (n + 1) + 9 * (n + 1) + 2 * nn);
 }
 
 cudaError_t launch_propose(const DevState& s, uint64_t seed, int64_t step, int slot_first, int count,
@@ -637,6 +681,7 @@ cudaError_t launch_propose(const DevState& s, uint64_t seed, int64_t step, int s
 __global__ void __launch_bounds__(DRAW_THREADS) k_draw(DevState s, uint64_t seed, int64_t step_arg, int N,
                                                        int K_arg, int burnin, int64_t M, int64_t total_steps) {
     extern __shared__ __align__(16) double dsm[];
+    MPCGS_TS(0);
     double* sC = dsm;  // [N+1] cumulative weights
     __shared__ double s_red[DRAW_THREADS / 32];
     __shared__ double s_max;
@@ -652,13 +697,12 @@ __global__ void __launch_bounds__(DRAW_THREADS) k_draw(DevState s, uint64_t seed
         r0[1] = s.gen[1];
         r0[2] = s.age[T];
         r0[3] = s.age[Par];
-        r0[4] = -1.0;
+        r0[4] = -1.0;  // read back only after later barriers
     }
-    __syncthreads();
     const int chunk = (nslots + DRAW_THREADS - 1) / DRAW_THREADS;
     const int i0 = tid * chunk, i1 = min(nslots, i0 + chunk);
     double mx = -CUDART_INF;
-    for (int i = i0; i < i1; ++i) mx = fmax(mx, s.rec[(size_t)i * REC]);
+    for (int i = i0; i < i1; ++i) mx = fmax(mx, i == 0 ? s.gen[0] : s.rec[(size_t)i * REC]);
 #pragma unroll
     for (int o = 16; o > 0; o >>= 1) mx = fmax(mx, __shfl_xor_sync(0xffffffffu, mx, o));
     if (lane == 0) s_red[wid] = mx;
@@ -684,6 +728,7 @@ __global__ void __launch_bounds__(DRAW_THREADS) k_draw(DevState s, uint64_t seed
         s_store = store;
     }
     __syncthreads();
+    MPCGS_TS(1);
     mx = s_max;
     if (!(mx > -CUDART_INF) || !(mx < CUDART_INF)) {  // all weights zero or NaN (S6)
         if (tid == 0) {
@@ -695,7 +740,7 @@ __global__ void __launch_bounds__(DRAW_THREADS) k_draw(DevState s, uint64_t seed
     // w_i = exp(logL_i - max): Eq. 31, proportional to P(D|G_i); inclusive scan in slot order
     double run = 0.0;
     for (int i = i0; i < i1; ++i) {
-        run += exp(s.rec[(size_t)i * REC] - mx);
+        run += exp((i == 0 ? s.gen[0] : s.rec[(size_t)i * REC]) - mx);
         sC[i] = run;
     }
     double x = run;
@@ -720,6 +765,7 @@ __global__ void __launch_bounds__(DRAW_THREADS) k_draw(DevState s, uint64_t seed
     const double before = (wid > 0 ? s_red[wid - 1] : 0.0) + (x - run);
     for (int i = i0; i < i1; ++i) sC[i] += before;
     __syncthreads();
+    MPCGS_TS(2);
     const int K = s_K;
     const double total = sC[N];
     const int64_t stored = s.counters[1];
@@ -743,6 +789,7 @@ __global__ void __launch_bounds__(DRAW_THREADS) k_draw(DevState s, uint64_t seed
         }
     }
     __syncthreads();
+    MPCGS_TS(3);
     // commit: the last draw generates the next proposal set (Fig. 12)
     const int I = K > 0 ? s.last_draws[K - 1] : 0;
     if (tid == 0 && I > 0) {
@@ -798,7 +845,15 @@ __global__ void __launch_bounds__(DRAW_THREADS) k_draw(DevState s, uint64_t seed
     // device loop: the next step's context, from the committed generator
     if (K_arg < 0 && step + 1 < total_steps) {
         __syncthreads();
+        MPCGS_TS(4);
         context_body<DRAW_THREADS>(s, seed, step + 1, dsm);
+        MPCGS_TS(11);
+#ifdef MPCGS_TIMESTAMPS
+        if (threadIdx.x == 0 && step == 2)
+            printf("draw: max %lld scan %lld draws %lld commit %lld | ctx: target %lld sort %lld dedupe %lld W %lld beta %lld rest %lld\n",
+                   g_ts[1] - g_ts[0], g_ts[2] - g_ts[1], g_ts[3] - g_ts[2], g_ts[4] - g_ts[3], g_ts[6] - g_ts[5],
+                   g_ts[7] - g_ts[6], g_ts[8] - g_ts[7], g_ts[9] - g_ts[8], g_ts[10] - g_ts[9], g_ts[11] - g_ts[10]);
+#endif
     }
 }
 
