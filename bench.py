@@ -168,6 +168,7 @@ def workload_config(args, wl):
     return {"workload": f"{args.workload}: {n} sequences x {L} bp, {wl['N']} proposals/step, theta0 {wl['theta0']}",
             "n_seq": n, "n_sites": L, "proposals_per_step": wl["N"], "theta0": wl["theta0"],
             "precision": args.precision, "l2": "flushed (256 MiB write) between timed steps",
+            "theta_true": getattr(args, "theta_true", 1.0),
             "parallelism": f"proposal-sharded x{args.gpus}", "init_tree": "synthetic true tree (ms-style)",
             "scoring": ("incremental rescoring (f2): partials/s counts the full-pruning equivalent n-1 nodes "
                         "per proposal and site" if getattr(args, "incremental", False) else "full pruning (5.2.2)")
@@ -183,6 +184,8 @@ def main():
     ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
     ap.add_argument("--workload", default="c5")
     ap.add_argument("--L", type=int, default=None)
+    ap.add_argument("--theta-true", type=float, default=1.0,
+                    help="theta of the simulated data (low values: few distinct columns, see --compress)")
     ap.add_argument("--n", type=int, default=None)
     ap.add_argument("--N", type=int, default=None)
     ap.add_argument("--precision", type=int, default=64, choices=[32, 64])
@@ -206,7 +209,7 @@ def main():
         over["n"] = args.n
     if args.N:
         over["N"] = args.N
-    wl = synth.workload(args.workload, **over)
+    wl = synth.workload(args.workload, theta_true=args.theta_true, **over)
     if args.impl == "reference":
         run_reference(args, wl, rank)
         return
