@@ -59,6 +59,12 @@ def lib():
         L.orc_default_rate.restype = c.c_double
         L.orc_transition.argtypes = [c.c_double, c.c_double, _f64p, _f64p]
         L.orc_check_tree.argtypes = [c.c_int, _i32p, _f64p]
+        L.orc_model_rate.argtypes = [c.c_int, c.c_double, _f64p]
+        L.orc_model_rate.restype = c.c_double
+        L.orc_transition_model.argtypes = [c.c_int, c.c_double, c.c_double, _f64p, _f64p]
+        L.orc_log_likelihood_model.argtypes = [c.c_int, c.c_double, c.c_int, c.c_int, _u8p, _i32p, _f64p,
+                                               _f64p, c.c_void_p]
+        L.orc_log_likelihood_model.restype = c.c_double
         L.orc_log_likelihood.argtypes = [c.c_int, c.c_int, _u8p, _i32p, _f64p, _f64p, c.c_double,
                                          c.c_void_p]
         L.orc_log_likelihood.restype = c.c_double
@@ -139,6 +145,28 @@ def transition(t, u, pi):
     P = np.zeros(16)
     lib().orc_transition(float(t), float(u), np.ascontiguousarray(pi, np.float64), P)
     return P.reshape(4, 4)
+
+
+MODELS = {"F81": 0, "F84": 1, "HKY85": 2}
+
+
+def model_rate(model, kappa, pi):
+    return lib().orc_model_rate(MODELS[model], float(kappa), np.ascontiguousarray(pi, np.float64))
+
+
+def transition_model(model, kappa, t, pi):
+    P = np.zeros(16)
+    lib().orc_transition_model(MODELS[model], float(kappa), float(t), np.ascontiguousarray(pi, np.float64), P)
+    return P.reshape(4, 4)
+
+
+def log_likelihood_model(model, kappa, codes, parent, age, pi):
+    """ln P(D|G) under F81 / F84 / HKY85, Eq. 19-22 in log space."""
+    codes = _codes(codes)
+    parent, age = _tree(parent, age)
+    n = (len(parent) + 1) // 2
+    return lib().orc_log_likelihood_model(MODELS[model], float(kappa), n, codes.shape[1], codes, parent, age,
+                                          np.ascontiguousarray(pi, np.float64), None)
 
 
 def check_tree(parent, age):

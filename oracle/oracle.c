@@ -109,6 +109,61 @@ void orc_transition(double t, double u, const double pi[4], double P[16]) {
         for (Y = 0; Y < 4; ++Y) P[X * 4 + Y] = (X == Y ? stay : 0.0) + (1.0 - stay) * pi[Y];
 }
 
+/* purine/pyrimidine group of a state and the group's total frequency */
+static int group_of(int X) { return (X == 0 || X == 2) ? 0 : 1; }
+static double group_freq(int X, const double pi[4]) {
+    return group_of(X) == 0 ? pi[0] + pi[2] : pi[1] + pi[3];
+}
+
+/* Rate mu that makes the expected number of substitutions per unit time 1. */
+double orc_model_rate(int model, double kappa, const double pi[4]) {
+    double sum = 0.0;
+    int X, Y;
+    if (model == 0) return orc_default_rate(pi);
+    for (X = 0; X < 4; ++X)
+        for (Y = 0; Y < 4; ++Y) {
+            double q;
+            if (X == Y) continue;
+            if (model == 1) /* F84: pi_Y (1 + kappa / Pi_g [same group]) */
+                q = pi[Y] * (1.0 + (group_of(X) == group_of(Y) ? kappa / group_freq(Y, pi) : 0.0));
+            else /* HKY85: kappa pi_Y for transitions, pi_Y for transversions */
+                q = (group_of(X) == group_of(Y) ? kappa : 1.0) * pi[Y];
+            sum += pi[X] * q;
+        }
+    return sum > 0.0 ? 1.0 / sum : 1.0;
+}
+
+void orc_transition_model(int model, double kappa, double t, const double pi[4], double P[16]) {
+    double mu = orc_model_rate(model, kappa, pi);
+    int X, Y;
+    if (model == 0) {
+        orc_transition(t, mu, pi, P);
+        return;
+    }
+    for (X = 0; X < 4; ++X)
+        for (Y = 0; Y < 4; ++Y) {
+            double PiY = group_freq(Y, pi), v;
+            int same = group_of(X) == group_of(Y);
+            if (model == 1) {
+                /* F84 (Felsenstein 1984): e^{-(1+k)mu t} d_XY
+                   + e^{-mu t}(1 - e^{-k mu t}) pi_Y / Pi_Y [same group] + (1 - e^{-mu t}) pi_Y */
+                v = (X == Y ? exp(-(1.0 + kappa) * mu * t) : 0.0) +
+                    (same ? exp(-mu * t) * (1.0 - exp(-kappa * mu * t)) * pi[Y] / PiY : 0.0) +
+                    (1.0 - exp(-mu * t)) * pi[Y];
+            } else {
+                /* HKY85 (Hasegawa, Kishino & Yano 1985), A_Y = 1 + Pi_Y (kappa - 1) */
+                double A = 1.0 + PiY * (kappa - 1.0);
+                if (X == Y)
+                    v = pi[Y] + pi[Y] * (1.0 / PiY - 1.0) * exp(-mu * t) + ((PiY - pi[Y]) / PiY) * exp(-mu * A * t);
+                else if (same)
+                    v = pi[Y] + pi[Y] * (1.0 / PiY - 1.0) * exp(-mu * t) - (pi[Y] / PiY) * exp(-mu * A * t);
+                else
+                    v = pi[Y] * (1.0 - exp(-mu * t));
+            }
+            P[X * 4 + Y] = v;
+        }
+}
+
 /* ------------------------------------------------------------------------- */
 /* Tree helpers.                                                              */
 /* ------------------------------------------------------------------------- */
@@ -215,8 +270,24 @@ static void prune_node(prune_work* w, int v, int site) {
     }
 }
 
+static double log_likelihood_impl(int model, double kappa, double u, int n, int L, const uint8_t* codes,
+                                  const int32_t* parent, const double* age, const double pi[4],
+                                  double* site_ll);
+
 double orc_log_likelihood(int n, int L, const uint8_t* codes, const int32_t* parent,
                           const double* age, const double pi[4], double u, double* site_ll) {
+    return log_likelihood_impl(0, 0.0, u, n, L, codes, parent, age, pi, site_ll);
+}
+
+double orc_log_likelihood_model(int model, double kappa, int n, int L, const uint8_t* codes,
+                                const int32_t* parent, const double* age, const double pi[4],
+                                double* site_ll) {
+    return log_likelihood_impl(model, kappa, 0.0, n, L, codes, parent, age, pi, site_ll);
+}
+
+static double log_likelihood_impl(int model, double kappa, double u, int n, int L, const uint8_t* codes,
+                                  const int32_t* parent, const double* age, const double pi[4],
+                                  double* site_ll) {
     int nn = 2 * n - 1, v, s, X;
     int32_t* left = (int32_t*)malloc(sizeof(int32_t) * (size_t)nn);
     int32_t* right = (int32_t*)malloc(sizeof(int32_t) * (size_t)nn);
@@ -230,7 +301,8 @@ double orc_log_likelihood(int n, int L, const uint8_t* codes, const int32_t* par
         double P[16];
         int i;
         if (parent[v] < 0) continue;
-        orc_transition(age[parent[v]] - age[v], u, pi, P);
+        if (model == 0) orc_transition(age[parent[v]] - age[v], u, pi, P);
+        else orc_transition_model(model, kappa, age[parent[v]] - age[v], pi, P);
         for (i = 0; i < 16; ++i) lnP[16 * v + i] = log(P[i]);
     }
     w.n = n;

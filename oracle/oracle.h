@@ -41,6 +41,17 @@ void orc_base_freqs(int n, int L, const uint8_t* codes, double pi[4]);
 double orc_default_rate(const double pi[4]);
 void orc_transition(double t, double u, const double pi[4], double P[16]);
 
+/* Model variants (seq-gen's F84 of the paper's data, L1508-1510,
+ * L1531-1533): model 0 = F81 (Eq. 20), 1 = F84, 2 = HKY85, transition /
+ * transversion parameter kappa; rates normalised to one expected substitution
+ * per unit time (reading S3).  Closed forms; states A, C, G, T = 0..3, purines
+ * {A, G}, pyrimidines {C, T}. */
+double orc_model_rate(int model, double kappa, const double pi[4]);
+void orc_transition_model(int model, double kappa, double t, const double pi[4], double P[16]);
+double orc_log_likelihood_model(int model, double kappa, int n, int L, const uint8_t* codes,
+                                const int32_t* parent, const double* age, const double pi[4],
+                                double* site_ll);
+
 /* Tree checks */
 int orc_check_tree(int n, const int32_t* parent, const double* age);
 

@@ -188,3 +188,60 @@ def test_theta_independence_of_data_likelihood(orc):
 def test_base_freqs_pooled(orc):
     codes = np.array([[0, 0, 1, 2], [3, 3, 3, 0]], np.uint8)
     assert np.allclose(orc.base_freqs(codes), [3 / 8, 1 / 8, 1 / 8, 3 / 8])
+
+
+# ------------------------------------------------------------------ f4: F84 / HKY85
+def _model_Q(model, kappa, pi):
+    """Rate matrix from the model's definition, normalised to mean rate 1."""
+    grp = [0, 1, 0, 1]                       # A, C, G, T: purines 0, pyrimidines 1
+    Pi = [pi[0] + pi[2], pi[1] + pi[3]]
+    Q = np.zeros((4, 4))
+    for i in range(4):
+        for j in range(4):
+            if i == j:
+                continue
+            same = grp[i] == grp[j]
+            if model == "F84":
+                Q[i, j] = pi[j] * (1 + (kappa / Pi[grp[j]] if same else 0.0))
+            else:  # HKY85
+                Q[i, j] = (kappa if same else 1.0) * pi[j]
+    np.fill_diagonal(Q, -Q.sum(axis=1))
+    return Q / -np.dot(pi, np.diag(Q))
+
+
+@pytest.mark.parametrize("model", ["F84", "HKY85"])
+@pytest.mark.parametrize("kappa", [0.5, 2.0, 7.3])
+def test_model_transition_is_expm(orc, model, kappa):
+    pi = np.array([0.35, 0.15, 0.2, 0.3])
+    Q = _model_Q(model, kappa, pi)
+    for t in [0.0, 1e-6, 0.05, 0.7, 3.0]:
+        P = orc.transition_model(model, kappa, t, pi)
+        assert np.allclose(P, scipy.linalg.expm(Q * t), rtol=1e-11, atol=1e-13)
+    # reductions to F81: F84 with kappa = 0, HKY85 with kappa = 1
+    u = orc.default_rate(pi)
+    assert np.allclose(orc.transition_model("F84", 0.0, 0.4, pi), orc.transition(0.4, u, pi), atol=1e-15)
+    assert np.allclose(orc.transition_model("HKY85", 1.0, 0.4, pi), orc.transition(0.4, u, pi), atol=1e-15)
+
+
+@pytest.mark.parametrize("model", ["F84", "HKY85"])
+def test_model_pruning_equals_brute_force(orc, model):
+    rng = np.random.default_rng(77)
+    n, kappa = 4, 3.0
+    parent, age = synth.shaped_tree(n, "random", rng, scale=0.3)
+    pi = np.array([0.3, 0.2, 0.15, 0.35])
+    codes = synth.random_alignment(n, 25, rng, pi)
+    Q = _model_Q(model, kappa, pi)
+    nn = 2 * n - 1
+    root = int(np.where(parent < 0)[0][0])
+    Pb = {v: scipy.linalg.expm(Q * (age[parent[v]] - age[v])) for v in range(nn) if parent[v] >= 0}
+    interior = list(range(n, nn))
+    total = np.zeros(codes.shape[1])
+    for assign in itertools.product(range(4), repeat=len(interior)):
+        st = dict(zip(interior, assign))
+        prob = np.full(codes.shape[1], pi[st[root]])
+        for v in range(nn):
+            if parent[v] >= 0:
+                prob = prob * (Pb[v][st[parent[v]], codes[v]] if v < n else Pb[v][st[parent[v]], st[v]])
+        total += prob
+    assert np.isclose(orc.log_likelihood_model(model, kappa, codes, parent, age, pi), np.log(total).sum(),
+                      rtol=1e-12)
