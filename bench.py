@@ -46,6 +46,13 @@ def flops_per_site(n: int) -> int:
     return 2 * n + 16 * (n - 2) + 4 * (n - 1)
 
 
+def flops_per_site_gm(n: int) -> int:
+    """Same under a general reversible model (F84 / HKY85): a tip
+    child is a column of P (0 flops), an internal child a 4x4 matrix-vector product
+    (16 mul + 12 add), node product 4."""
+    return 28 * (n - 2) + 4 * (n - 1)
+
+
 def peaks():
     mp = {}
     try:
@@ -105,7 +112,13 @@ def traffic_from_profiles(tag: str):
         return None
 
 
-def cpu_oracle_sample(wl, seconds: float, n_prop: int = 1):
+def oracle_gen_logL(oracle, codes, parent, age, pi, u, model, kappa):
+    if model == "F81":
+        return oracle.log_likelihood(codes, parent, age, pi, u)
+    return oracle.log_likelihood_model(model, kappa, codes, parent, age, pi)
+
+
+def cpu_oracle_sample(wl, seconds: float, n_prop: int = 1, model="F81", kappa=0.0):
     """Time the oracle's GMH step on the same workload (bounded: n_prop proposals)."""
     import oracle
 
@@ -113,11 +126,12 @@ def cpu_oracle_sample(wl, seconds: float, n_prop: int = 1):
     pi = oracle.base_freqs(codes)
     u = oracle.default_rate(pi)
     parent, age = wl["true_parent"], wl["true_age"]
-    gl = oracle.log_likelihood(codes, parent, age, pi, u)
+    gl = oracle_gen_logL(oracle, codes, parent, age, pi, u, model, kappa)
     n, L = codes.shape
     steps, t0 = 0, time.perf_counter()
     while True:
-        tr = oracle.gmh_step(codes, pi, u, wl["theta0"], n_prop, n_prop, wl["chain_seed"], steps, parent, age, gl)
+        tr = oracle.gmh_step(codes, pi, u, wl["theta0"], n_prop, n_prop, wl["chain_seed"], steps, parent, age, gl,
+                             model=model, kappa=kappa)
         parent, age, gl = tr["parent"], tr["age"], tr["gen_logL"]
         steps += 1
         if time.perf_counter() - t0 >= seconds:
@@ -137,15 +151,16 @@ def run_reference(args, wl, rank):
     pi = oracle.base_freqs(codes)
     u = oracle.default_rate(pi)
     parent, age = wl["true_parent"], wl["true_age"]
-    gl = oracle.log_likelihood(codes, parent, age, pi, u)
+    gl = oracle_gen_logL(oracle, codes, parent, age, pi, u, args.model, args.kappa)
     n_prop = 1
+    mk = dict(model=args.model, kappa=args.kappa)
     for s in range(args.warmup):
-        tr = oracle.gmh_step(codes, pi, u, wl["theta0"], n_prop, n_prop, wl["chain_seed"], s, parent, age, gl)
+        tr = oracle.gmh_step(codes, pi, u, wl["theta0"], n_prop, n_prop, wl["chain_seed"], s, parent, age, gl, **mk)
         parent, age, gl = tr["parent"], tr["age"], tr["gen_logL"]
     t0 = time.perf_counter()
     for s in range(args.steps):
         tr = oracle.gmh_step(codes, pi, u, wl["theta0"], n_prop, n_prop, wl["chain_seed"], args.warmup + s,
-                             parent, age, gl)
+                             parent, age, gl, **mk)
         parent, age, gl = tr["parent"], tr["age"], tr["gen_logL"]
     dt = time.perf_counter() - t0
     partials = args.steps * n_prop * L * (n - 1)
@@ -173,7 +188,8 @@ def workload_config(args, wl):
             "scoring": ("incremental rescoring (f2): partials/s counts the full-pruning equivalent n-1 nodes "
                         "per proposal and site" if getattr(args, "incremental", False) else "full pruning (5.2.2)")
             + ("; compressed site patterns (f3): partials/s counts all L columns" if getattr(args, "compress", False)
-               else "")}
+               else ""),
+            "model": args.model + ("" if args.model == "F81" else f" (kappa {args.kappa}; SURVEY 8(f) f4)")}
 
 
 def main():
@@ -196,6 +212,9 @@ def main():
                     help="score distinct alignment columns weighted by count (SURVEY 8(f) f3)")
     ap.add_argument("--incremental", action="store_true",
                     help="score proposals by incremental rescoring (SURVEY 8(f) f2) instead of full pruning")
+    ap.add_argument("--model", default="F81", choices=["F81", "F84", "HKY85"],
+                    help="substitution model (F84 / HKY85: SURVEY 8(f) f4)")
+    ap.add_argument("--kappa", type=float, default=2.0, help="F84 / HKY85 transition/transversion parameter")
     args = ap.parse_args()
     args.warmup = max(args.warmup, 3)
 
@@ -250,7 +269,8 @@ def main():
 
     ctx = P.Context(rows, wl["theta0"], precision=args.precision, max_proposals=N, max_samples=N * total_steps,
                     init_tree=(wl["true_parent"], wl["true_age"]), rank=rank, world=world, nccl_id=nccl_id,
-                    stream=stream, incremental=args.incremental, compress_patterns=args.compress)
+                    stream=stream, incremental=args.incremental, compress_patterns=args.compress,
+                    model=args.model, kappa=args.kappa)
     # warm-up (untimed): W steps
     ctx.mpcgs_sample(N, N * args.warmup, wl["chain_seed"])
     ctx.mpcgs_set_timing(3)   # per-step + per-prune CUDA events, L2 flush between steps
@@ -271,12 +291,15 @@ def main():
     # roofline of the dominant kernel (prune): algorithmic flops per launch / mean launch time
     pk, mhz, mp = peaks()
     local_trees = N // world
-    flops_launch = local_trees * L * flops_per_site(n)
+    gm = args.model != "F81"
+    flops_launch = local_trees * L * (flops_per_site_gm(n) if gm else flops_per_site(n))
     prune_avg_s = (prune_ms / 1e3) / args.steps
     achieved = flops_launch / prune_avg_s / 1e12
     roof = {"bound": "alu", "achieved": achieved, "peak": pk[args.precision], "unit": "TFLOP/s",
-            "frac": achieved / pk[args.precision], "traffic": traffic_from_profiles(f"{args.workload}_fp{args.precision}"),
-            "kernel": "k_prune", "prune_share_of_step": prune_ms / loop_ms,
+            "frac": achieved / pk[args.precision],
+            "traffic": traffic_from_profiles(f"{args.workload}_fp{args.precision}" + (f"_{args.model}" if gm else "")),
+            "kernel": "k_prune (flat, general model) + k_pmat" if gm else "k_prune_tab",
+            "prune_share_of_step": prune_ms / loop_ms,
             "peak_source": f"derived: 148 SM x {'64 FP64' if args.precision == 64 else '128 FP32'} FMA lanes x 2 x "
                            f"{mhz:.0f} MHz (MEASURED_PEAKS sm_max_mhz)",
             "partials_per_s_prune_only": N * L * (n - 1) / (prune_avg_s * world) if world == 1 else
@@ -290,7 +313,8 @@ def main():
         t0 = time.perf_counter()
         ctx2 = P.Context(rows, wl["theta0"], precision=args.precision, max_proposals=N, max_samples=N * args.steps,
                          init_tree=(wl["true_parent"], wl["true_age"]), rank=rank, world=world,
-                         nccl_id=fresh_nccl_id(), stream=stream, incremental=args.incremental)
+                         nccl_id=fresh_nccl_id(), stream=stream, incremental=args.incremental,
+                         compress_patterns=args.compress, model=args.model, kappa=args.kappa)
         ctx2.mpcgs_sample(N, N * args.steps, wl["chain_seed"] + 1)
         smp = ctx2.mpcgs_get_samples()
         barrier()
@@ -309,7 +333,7 @@ def main():
     # the same workload scored by incremental rescoring, reported
     # beside the full-pruning headline (its partials/s counts n-1 nodes per proposal)
     incr = None
-    if not args.incremental and not args.no_incremental_block:
+    if not args.incremental and not args.no_incremental_block and not gm:
         ctx3 = P.Context(rows, wl["theta0"], precision=args.precision, max_proposals=N,
                          max_samples=N * (args.warmup + args.steps), init_tree=(wl["true_parent"], wl["true_age"]),
                          rank=rank, world=world, nccl_id=fresh_nccl_id(), stream=stream, incremental=True)
@@ -330,7 +354,7 @@ def main():
 
     cpu = None
     if rank == 0 and world == 1 and args.cpu_seconds > 0:
-        v, st, dt = cpu_oracle_sample(wl, args.cpu_seconds)
+        v, st, dt = cpu_oracle_sample(wl, args.cpu_seconds, model=args.model, kappa=args.kappa)
         cpu = {"value": v, "unit": UNIT, "cores": 1, "kind": "oracle",
                "sample": f"{st} oracle GMH steps with 1 proposal each over all {L} sites ({dt:.1f} s)"}
 

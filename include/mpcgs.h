@@ -93,7 +93,17 @@ typedef struct {
                               recomputes only T, Par and the ancestors of Par (L1390-1398) */
     int32_t compress_patterns; /* 1: score each distinct alignment column once, weighted by its
                               count (exact by site independence, L714-716) */
+    int32_t model;         /* substitution model: MPCGS_MODEL_F81 (Eq. 20, the
+                              paper's), MPCGS_MODEL_F84 (seq-gen's model of the paper's data,
+                              L1508-1510) or MPCGS_MODEL_HKY85.  F84 / HKY85: rates normalised to
+                              one expected substitution per unit time (mu is ignored), every
+                              pi > 0, incremental = 0 (else MPCGS_E_ARG) */
+    double kappa;          /* transition/transversion parameter of F84 / HKY85 (>= 0) */
 } mpcgs_config;
+
+#define MPCGS_MODEL_F81 0
+#define MPCGS_MODEL_F84 1
+#define MPCGS_MODEL_HKY85 2
 
 /* [host-only] Fill cfg with defaults: empirical pi, default u, precision 64, burn-in 0,
  * max_proposals 1024, max_samples 1<<20, world 1. */
@@ -105,6 +115,17 @@ size_t mpcgs_workspace_bytes(int32_t n_seq, int32_t n_sites, int32_t max_proposa
 /* [host-only] Same, with incremental rescoring on (incremental != 0). */
 size_t mpcgs_workspace_bytes_ex(int32_t n_seq, int32_t n_sites, int32_t max_proposals,
                                 int64_t max_samples, int32_t precision, int32_t incremental);
+
+/* [host-only] Same, for every capacity / option of cfg (precision, max_proposals,
+ * max_samples, incremental, model).  0 on invalid arguments. */
+size_t mpcgs_workspace_bytes_cfg(int32_t n_seq, int32_t n_sites, const mpcgs_config* cfg);
+
+/* [host-only] Transition matrix P(t) (row-major, P[i*4+j] = Pr(j at the child | i at the
+ * parent), states A,C,G,T) as the kernels form it: F81 by Eq. 20 (L696-699) with rate mu;
+ * F84 / HKY85 from the eigen-decomposition of the normalised rate matrix (mu unused).
+ * pi: host [4].  MPCGS_E_ARG on a bad model / kappa / t, or pi <= 0 for F84 / HKY85. */
+mpcgs_status mpcgs_transition(int32_t model, double kappa, const double* pi, double mu, double t,
+                              double* P);
 
 /* Create a context: validate and copy the alignment, compute pi and u, build G0
  * (init_parent/init_age, else UPGMA), upload everything to the device and score

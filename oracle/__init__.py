@@ -82,6 +82,9 @@ def lib():
         L.orc_gmh_step.argtypes = [c.c_int, c.c_int, _u8p, _f64p, c.c_double, c.c_double, c.c_int,
                                    c.c_int, c.c_uint64, c.c_uint32, _i32p, _f64p, _f64p, _i32p,
                                    _f64p, _f64p, _f64p, _i32p, _i32p, _i32p, _i32p]
+        L.orc_gmh_step_model.argtypes = [c.c_int, c.c_double, c.c_int, c.c_int, _u8p, _f64p, c.c_double,
+                                         c.c_int, c.c_int, c.c_uint64, c.c_uint32, _i32p, _f64p, _f64p,
+                                         _i32p, _f64p, _f64p, _f64p, _i32p, _i32p, _i32p, _i32p]
         L.orc_run_chain.argtypes = [c.c_int, c.c_int, _u8p, _f64p, c.c_double, c.c_double,
                                     c.c_int, c.c_int, c.c_int, c.c_uint64, _i32p, _f64p, _f64p,
                                     _f64p, _i64p, _i32p, _i32p]
@@ -245,8 +248,9 @@ def draw(cum, u):
     return i, bool(flag[0])
 
 
-def gmh_step(codes, pi, u, theta0, N, K, seed, step, parent, age, gen_logL):
-    """One GMH step (Alg. 1, Fig. 12). Returns a dict trace and the new generator."""
+def gmh_step(codes, pi, u, theta0, N, K, seed, step, parent, age, gen_logL, model="F81", kappa=0.0):
+    """One GMH step (Alg. 1, Fig. 12). Returns a dict trace and the new generator.
+    model "F84" / "HKY85": P(D|G) under that model, u unused."""
     codes = _codes(codes)
     parent, age = _tree(parent, age)
     parent, age = parent.copy(), age.copy()
@@ -260,9 +264,15 @@ def gmh_step(codes, pi, u, theta0, N, K, seed, step, parent, age, gen_logL):
     sflag = np.zeros(N + 1, np.int32)
     draws = np.zeros(max(K, 1), np.int32)
     dflag = np.zeros(max(K, 1), np.int32)
-    _chk(lib().orc_gmh_step(n, codes.shape[1], codes, np.ascontiguousarray(pi, np.float64),
-                            float(u), theta0, N, K, seed, step, parent, age, gl, tgt, logL, S, t12,
-                            pair, sflag, draws, dflag))
+    m = MODELS[model] if isinstance(model, str) else int(model)
+    if m == 0:
+        _chk(lib().orc_gmh_step(n, codes.shape[1], codes, np.ascontiguousarray(pi, np.float64),
+                                float(u), theta0, N, K, seed, step, parent, age, gl, tgt, logL, S, t12,
+                                pair, sflag, draws, dflag))
+    else:
+        _chk(lib().orc_gmh_step_model(m, float(kappa), n, codes.shape[1], codes,
+                                      np.ascontiguousarray(pi, np.float64), theta0, N, K, seed, step,
+                                      parent, age, gl, tgt, logL, S, t12, pair, sflag, draws, dflag))
     return dict(target=int(tgt[0]), logL=logL, S=S, t12=t12.reshape(N + 1, 2), pair=pair,
                 slot_flag=sflag.astype(bool), draws=draws[:K], draw_flag=dflag[:K].astype(bool),
                 parent=parent, age=age, gen_logL=float(gl[0]))

@@ -805,11 +805,11 @@ int orc_draw(int nslots, const double* cum, double u, int32_t* flag) {
     return nslots - 1;
 }
 
-int orc_gmh_step(int n, int L, const uint8_t* codes, const double pi[4], double u,
-                 double theta0, int N, int K, uint64_t seed, uint32_t step,
-                 int32_t* gen_parent, double* gen_age, double* gen_logL,
-                 int32_t* out_target, double* slot_logL, double* slot_S, double* slot_t12,
-                 int32_t* slot_pair, int32_t* slot_flag, int32_t* draws, int32_t* draw_flag) {
+static int gmh_step_impl(int model, double kappa, int n, int L, const uint8_t* codes,
+                         const double pi[4], double u, double theta0, int N, int K, uint64_t seed,
+                         uint32_t step, int32_t* gen_parent, double* gen_age, double* gen_logL,
+                         int32_t* out_target, double* slot_logL, double* slot_S, double* slot_t12,
+                         int32_t* slot_pair, int32_t* slot_flag, int32_t* draws, int32_t* draw_flag) {
     int nn = 2 * n - 1, i, d, rc, last = 0;
     int32_t* par_all = (int32_t*)malloc(sizeof(int32_t) * (size_t)nn * (size_t)(N + 1));
     double* age_all = (double*)malloc(sizeof(double) * (size_t)nn * (size_t)(N + 1));
@@ -835,7 +835,8 @@ int orc_gmh_step(int n, int L, const uint8_t* codes, const double pi[4], double 
         rc = propose_from_ctx(n, gen_parent, gen_age, &cx, seed, step, (uint32_t)i, pp, aa,
                               slot_t12 + 2 * i, slot_pair + i, slot_flag + i);
         if (rc != ORC_OK) goto done;
-        slot_logL[i] = orc_log_likelihood(n, L, codes, pp, aa, pi, u, NULL);
+        slot_logL[i] = model == 0 ? orc_log_likelihood(n, L, codes, pp, aa, pi, u, NULL)
+                                  : orc_log_likelihood_model(model, kappa, n, L, codes, pp, aa, pi, NULL);
         slot_S[i] = orc_coalescent_S(n, aa);
     }
     rc = orc_weights(N + 1, slot_logL, w, cum);
@@ -856,6 +857,29 @@ done:
     free(w);
     free(cum);
     return rc;
+}
+
+int orc_gmh_step(int n, int L, const uint8_t* codes, const double pi[4], double u,
+                 double theta0, int N, int K, uint64_t seed, uint32_t step,
+                 int32_t* gen_parent, double* gen_age, double* gen_logL,
+                 int32_t* out_target, double* slot_logL, double* slot_S, double* slot_t12,
+                 int32_t* slot_pair, int32_t* slot_flag, int32_t* draws, int32_t* draw_flag) {
+    return gmh_step_impl(0, 0.0, n, L, codes, pi, u, theta0, N, K, seed, step, gen_parent, gen_age,
+                         gen_logL, out_target, slot_logL, slot_S, slot_t12, slot_pair, slot_flag,
+                         draws, draw_flag);
+}
+
+/* The same step with P(D|G) under model 1 (F84) or 2 (HKY85): only the
+   likelihood of Eq. 22 changes; proposals, weights and draws are those of Alg. 1. */
+int orc_gmh_step_model(int model, double kappa, int n, int L, const uint8_t* codes,
+                       const double pi[4], double theta0, int N, int K, uint64_t seed,
+                       uint32_t step, int32_t* gen_parent, double* gen_age, double* gen_logL,
+                       int32_t* out_target, double* slot_logL, double* slot_S, double* slot_t12,
+                       int32_t* slot_pair, int32_t* slot_flag, int32_t* draws, int32_t* draw_flag) {
+    if (model < 0 || model > 2) return ORC_E_ARG;
+    return gmh_step_impl(model, kappa, n, L, codes, pi, orc_model_rate(model, kappa, pi), theta0, N,
+                         K, seed, step, gen_parent, gen_age, gen_logL, out_target, slot_logL,
+                         slot_S, slot_t12, slot_pair, slot_flag, draws, draw_flag);
 }
 
 int orc_run_chain(int n, int L, const uint8_t* codes, const double pi[4], double u,

@@ -87,6 +87,13 @@ int orc_gmh_step(int n, int L, const uint8_t* codes, const double pi[4], double 
                  int32_t* out_target, double* slot_logL, double* slot_S, double* slot_t12,
                  int32_t* slot_pair, int32_t* slot_flag, int32_t* draws, int32_t* draw_flag);
 
+/* Same step with P(D|G) under model 1 (F84) / 2 (HKY85), kappa */
+int orc_gmh_step_model(int model, double kappa, int n, int L, const uint8_t* codes,
+                       const double pi[4], double theta0, int N, int K, uint64_t seed,
+                       uint32_t step, int32_t* gen_parent, double* gen_age, double* gen_logL,
+                       int32_t* out_target, double* slot_logL, double* slot_S, double* slot_t12,
+                       int32_t* slot_pair, int32_t* slot_flag, int32_t* draws, int32_t* draw_flag);
+
 /* Burn-in + sampling chain (Fig. 11/12, Alg. 1) */
 int orc_run_chain(int n, int L, const uint8_t* codes, const double pi[4], double u,
                   double theta0, int N, int burnin, int M, uint64_t seed,

@@ -147,6 +147,10 @@ struct DevState {
     double pi[4];
     double u;       // F81 rate (S3)
     double theta0;  // driving value
+    int model;             // 0: F81 (Eq. 20), branch data e/em.  1: general reversible model
+                           // (F84, HKY85: SURVEY 8(f) f4), branch data (t, 0), P(t) from gm
+    const double* gm;      // [36] ev[4], V[16], W[16]: P(t) = V diag(exp(ev t)) W (model 1)
+    void* sched_P;         // [Nmax][nops][32] P of each op's two children (model 1)
     const uint8_t* codes;  // [n][Lpad], 0..3
     const double* site_w;  // [L] pattern counts when sites are compressed patterns (f3), else nullptr
     // generator (chain state)
@@ -193,6 +197,33 @@ struct DevState {
     int32_t* csib;      // [n]
     int32_t* gen_order; // [n-1] interior nodes children-first (full partial recompute)
 };
+
+// Transition matrix of a general reversible model from its eigen-decomposition
+// gm = {ev[4], V[16], W[16]}: P_ij(t) = sum_k V_ik exp(ev_k t) W_kj (row i = the
+// state at the parent end).  Entries are clamped at 0 (true P(t) >= 0; the
+// eigen route leaves rounding-size negatives near t = 0).
+__host__ __device__ inline void pmat(const double* gm, double t, double* P) {
+    double ex[4];
+    for (int k = 0; k < 4; ++k) ex[k] = exp(gm[k] * t);
+    for (int i = 0; i < 4; ++i)
+        for (int j = 0; j < 4; ++j) {
+            double v = 0.0;
+            for (int k = 0; k < 4; ++k) v = fma(gm[4 + i * 4 + k] * ex[k], gm[20 + k * 4 + j], v);
+            P[i * 4 + j] = v > 0.0 ? v : 0.0;
+        }
+}
+
+// Branch data of a branch of length t: F81 {e, em} = {exp(-u t), -expm1(-u t)}
+// (Eq. 20); general model {t, 0} (P(t) is formed per op by k_pmat).
+__host__ __device__ __forceinline__ void branch_data(int model, double u, double t, double& e, double& em) {
+    if (model) {
+        e = t;
+        em = 0.0;
+    } else {
+        e = exp(-u * t);
+        em = -expm1(-u * t);
+    }
+}
 
 // counters[2] status bits
 constexpr int64_t STATUS_NUMERIC = 1;

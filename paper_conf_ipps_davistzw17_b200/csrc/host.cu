@@ -60,6 +60,8 @@ struct mpcgs_ctx {
     int n = 0, L = 0, nn = 0, Lpad = 0, nops = 0, depth = 0, precision = 64;
     int world = 1, rank = 0, burnin = 0;
     bool incremental = false;
+    int model = 0;           // MPCGS_MODEL_*
+    double kappa = 0.0;
     int L_orig = 0;          // alignment columns (L = scored sites: patterns if compressed)
     int Nmax = 0;
     int64_t Mmax = 0;
@@ -112,6 +114,7 @@ mpcgs_status fail(mpcgs_ctx* c, mpcgs_status st, const std::string& msg) {
 // ------------------------------------------------------------ workspace layout
 struct Layout {
     size_t codes, codes2, parent, left, right, need, age, e, em, gen, ctx_i, ctx_d, tau, len, lcnt, entry, omega, fixed;
+    size_t gm, sched_P;
     size_t tree_need, rec, sched_op, sched_e, tile_part, tile_cnt, sS, sL, sStep, sSlot, counters, last_draws, theta_buf,
         theta_cnt, score_out, site_w, GL, GE, path, pathsib, cpath, csib, ixyz, iee, cinfo, gen_order, total;
     int tiles_max;
@@ -122,7 +125,7 @@ size_t al(size_t x) { return (x + 255) & ~(size_t)255; }
 // 2-bit packed tip codes, 16 sites per 32-bit word, rows padded past the last tile
 int codes2_words(int L) { return ((L + 4096 + 63) / 64) * 4; }
 
-Layout layout(int n, int L, int Nmax, int64_t Mmax, int precision, int incremental = 0) {
+Layout layout(int n, int L, int Nmax, int64_t Mmax, int precision, int incremental = 0, int model = 0) {
     Layout y{};
     const int nn = 2 * n - 1, nops = n - 1;
     const int Lpad = (L + 15) & ~15;
@@ -179,8 +182,87 @@ Layout layout(int n, int L, int Nmax, int64_t Mmax, int precision, int increment
     y.iee = take(80 * (size_t)Nmax);
     y.cinfo = take(32);
     y.gen_order = take(4 * (size_t)n);
+    y.gm = take(model ? 8 * 36 : 0);
+    y.sched_P = take(model ? 16 * tsz * 2 * (size_t)Nmax * nops : 0);
     y.total = o;
     return y;
+}
+
+// ------------------------------------------------------------ substitution models (f4)
+// Rate matrix of the model (i != j; rows sum to 0), scaled to one expected
+// substitution per unit time (S3).  Purines A, G = 0, 2; pyrimidines C, T = 1, 3.
+//   F84   (Felsenstein 1984): q_ij = pi_j (1 + kappa / Pi_{g(j)} [g(i) = g(j)])
+//   HKY85 (Hasegawa, Kishino & Yano 1985): q_ij = pi_j (kappa [g(i) = g(j)] + [g(i) != g(j)])
+void rate_matrix(int model, double kappa, const double pi[4], double Q[16]) {
+    auto grp = [](int x) { return x & 1; };
+    const double Pi[2] = {pi[0] + pi[2], pi[1] + pi[3]};
+    double flux = 0.0;
+    for (int i = 0; i < 4; ++i) {
+        double row = 0.0;
+        for (int j = 0; j < 4; ++j) {
+            if (i == j) continue;
+            const bool ts = grp(i) == grp(j);
+            double q;
+            if (model == MPCGS_MODEL_F84) q = pi[j] * (1.0 + (ts ? kappa / Pi[grp(j)] : 0.0));
+            else if (model == MPCGS_MODEL_HKY85) q = pi[j] * (ts ? kappa : 1.0);
+            else q = pi[j];  // F81
+            Q[i * 4 + j] = q;
+            row += q;
+        }
+        Q[i * 4 + i] = -row;
+        flux += pi[i] * row;
+    }
+    const double scale = flux > 0.0 ? 1.0 / flux : 1.0;
+    for (int k = 0; k < 16; ++k) Q[k] *= scale;
+}
+
+// Eigen-system of a reversible Q: S = D^1/2 Q D^-1/2 (D = diag pi) is symmetric;
+// cyclic Jacobi gives S = U diag(ev) U^T, so P(t) = e^{Qt} = V diag(e^{ev t}) W with
+// V = D^-1/2 U and W = U^T D^1/2.  gm = {ev[4], V[16], W[16]}.  Needs pi > 0.
+void eigen_system(const double Q[16], const double pi[4], double gm[36]) {
+    double A[16], U[16];
+    for (int i = 0; i < 4; ++i)
+        for (int j = 0; j < 4; ++j) {
+            A[i * 4 + j] = std::sqrt(pi[i] / pi[j]) * Q[i * 4 + j];
+            U[i * 4 + j] = i == j ? 1.0 : 0.0;
+        }
+    for (int i = 0; i < 4; ++i)  // exact symmetry (rounding)
+        for (int j = i + 1; j < 4; ++j) A[i * 4 + j] = A[j * 4 + i] = 0.5 * (A[i * 4 + j] + A[j * 4 + i]);
+    for (int sweep = 0; sweep < 64; ++sweep) {
+        double off = 0.0;
+        for (int i = 0; i < 4; ++i)
+            for (int j = i + 1; j < 4; ++j) off += A[i * 4 + j] * A[i * 4 + j];
+        if (off < 1e-300) break;
+        for (int p = 0; p < 4; ++p)
+            for (int q = p + 1; q < 4; ++q) {
+                const double apq = A[p * 4 + q];
+                if (apq == 0.0) continue;
+                const double th = (A[q * 4 + q] - A[p * 4 + p]) / (2.0 * apq);
+                const double t = (th >= 0.0 ? 1.0 : -1.0) / (std::fabs(th) + std::sqrt(th * th + 1.0));
+                const double cs = 1.0 / std::sqrt(t * t + 1.0), sn = t * cs;
+                for (int k = 0; k < 4; ++k) {  // A <- J^T A J (columns, then rows)
+                    const double akp = A[k * 4 + p], akq = A[k * 4 + q];
+                    A[k * 4 + p] = cs * akp - sn * akq;
+                    A[k * 4 + q] = sn * akp + cs * akq;
+                }
+                for (int k = 0; k < 4; ++k) {
+                    const double apk = A[p * 4 + k], aqk = A[q * 4 + k];
+                    A[p * 4 + k] = cs * apk - sn * aqk;
+                    A[q * 4 + k] = sn * apk + cs * aqk;
+                }
+                for (int k = 0; k < 4; ++k) {  // U <- U J
+                    const double ukp = U[k * 4 + p], ukq = U[k * 4 + q];
+                    U[k * 4 + p] = cs * ukp - sn * ukq;
+                    U[k * 4 + q] = sn * ukp + cs * ukq;
+                }
+            }
+    }
+    for (int k = 0; k < 4; ++k) gm[k] = std::min(A[k * 4 + k], 0.0);  // Q is negative semi-definite
+    for (int i = 0; i < 4; ++i)
+        for (int k = 0; k < 4; ++k) {
+            gm[4 + i * 4 + k] = U[i * 4 + k] / std::sqrt(pi[i]);
+            gm[20 + k * 4 + i] = U[i * 4 + k] * std::sqrt(pi[i]);
+        }
 }
 
 // ------------------------------------------------------------ host tree helpers
@@ -221,7 +303,7 @@ struct HostTree {
 };
 
 // children (lower id first), Sethi-Ullman needs (post-order), branch factors
-void host_tree(int n, const int32_t* parent, const double* age, double u, HostTree& t) {
+void host_tree(int n, const int32_t* parent, const double* age, double u, HostTree& t, int model = 0) {
     const int nn = 2 * n - 1;
     t.left.assign(nn, -1);
     t.right.assign(nn, -1);
@@ -234,9 +316,7 @@ void host_tree(int n, const int32_t* parent, const double* age, double u, HostTr
         if (t.left[p] < 0) t.left[p] = v;
         else if (v < t.left[p]) { t.right[p] = t.left[p]; t.left[p] = v; }
         else t.right[p] = v;
-        const double len = age[p] - age[v];
-        t.e[v] = std::exp(-u * len);
-        t.em[v] = -std::expm1(-u * len);
+        branch_data(model, u, age[p] - age[v], t.e[v], t.em[v]);
     }
     // post-order by an explicit stack
     std::vector<int> st;
@@ -361,6 +441,8 @@ PruneArgs prune_args(mpcgs_ctx* c, int ntrees_global, double* out, int out_first
     for (int i = 0; i < 4; ++i) a.pi[i] = c->s.pi[i];
     a.sched_op = c->s.sched_op;
     a.sched_e = c->s.sched_e;
+    a.gm = c->model ? c->s.gm : nullptr;
+    a.sched_P = c->s.sched_P;
     prune_tiling(c->n, c->L, ntrees_global, c->precision, a.tiles, a.sites_per_cta);
     a.tree_need = c->s.tree_need;
     a.tile_part = c->s.tile_part;
@@ -396,7 +478,7 @@ mpcgs_status score_batch(mpcgs_ctx* c, int count, const int32_t* parent, const d
         if (check_tree(n, parent + (size_t)t * nn, age + (size_t)t * nn, why))
             return fail(c, MPCGS_E_ARG, "tree " + std::to_string(t) + ": " + why);
         HostTree ht;
-        host_tree(n, parent + (size_t)t * nn, age + (size_t)t * nn, c->s.u, ht);
+        host_tree(n, parent + (size_t)t * nn, age + (size_t)t * nn, c->s.u, ht, c->model);
         int d = c->precision == 32 ? host_schedule<float>(n, ht, ops.data() + (size_t)t * nops,
                                                           e4.data() + (size_t)t * nops * 4)
                                    : host_schedule<double>(n, ht, ops.data() + (size_t)t * nops,
@@ -422,7 +504,7 @@ mpcgs_status upload_state(mpcgs_ctx* c, const int32_t* parent, const double* age
     std::string why;
     if (check_tree(n, parent, age, why)) return fail(c, MPCGS_E_ARG, "generator: " + why);
     HostTree ht;
-    host_tree(n, parent, age, c->s.u, ht);
+    host_tree(n, parent, age, c->s.u, ht, c->model);
     if (ht.need[ht.root] > c->depth) return fail(c, MPCGS_E_ARG, "tree needs more registers than compiled");
     double logL = 0.0;
     mpcgs_status st = score_batch(c, 1, parent, age, &logL);
@@ -535,6 +617,33 @@ size_t mpcgs_workspace_bytes_ex(int32_t n_seq, int32_t n_sites, int32_t max_prop
                                 int32_t precision, int32_t incremental) {
     if (n_seq < 2 || n_sites < 1 || max_proposals < 1 || max_samples < 0) return 0;
     return layout(n_seq, n_sites, max_proposals, max_samples, precision, incremental != 0).total;
+}
+
+size_t mpcgs_workspace_bytes_cfg(int32_t n_seq, int32_t n_sites, const mpcgs_config* cfg) {
+    if (!cfg || n_seq < 2 || n_sites < 1 || cfg->max_proposals < 1 || cfg->max_samples < 0) return 0;
+    return layout(n_seq, n_sites, cfg->max_proposals, cfg->max_samples, cfg->precision, cfg->incremental != 0,
+                  cfg->model)
+        .total;
+}
+
+mpcgs_status mpcgs_transition(int32_t model, double kappa, const double* pi, double mu, double t, double* P) {
+    if (!pi || !P || !(t >= 0.0) || !std::isfinite(t)) return MPCGS_E_ARG;
+    if (model == MPCGS_MODEL_F81) {
+        double e, em;
+        branch_data(0, mu, t, e, em);
+        for (int i = 0; i < 4; ++i)
+            for (int j = 0; j < 4; ++j) P[i * 4 + j] = (i == j ? e : 0.0) + em * pi[j];
+        return MPCGS_OK;
+    }
+    if ((model != MPCGS_MODEL_F84 && model != MPCGS_MODEL_HKY85) || !(kappa >= 0.0) || !std::isfinite(kappa))
+        return MPCGS_E_ARG;
+    for (int i = 0; i < 4; ++i)
+        if (!(pi[i] > 0.0)) return MPCGS_E_ARG;
+    double Q[16], gm[36];
+    rate_matrix(model, kappa, pi, Q);
+    eigen_system(Q, pi, gm);
+    pmat(gm, t, P);
+    return MPCGS_OK;
 }
 
 void mpcgs_philox(const uint32_t ctr[4], const uint32_t key[2], uint32_t out[4]) {
@@ -691,6 +800,26 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
     }
     double sq = pi[0] * pi[0] + pi[1] * pi[1] + pi[2] * pi[2] + pi[3] * pi[3];
     double u = cfg->mu > 0.0 ? cfg->mu : (sq < 1.0 ? 1.0 / (1.0 - sq) : 1.0);
+    // substitution model: F81 unless F84 / HKY85 is asked for
+    c->model = cfg->model;
+    c->kappa = cfg->kappa;
+    double gm[36] = {0};
+    if (c->model != MPCGS_MODEL_F81) {
+        const char* why = nullptr;
+        if (c->model != MPCGS_MODEL_F84 && c->model != MPCGS_MODEL_HKY85) why = "unknown substitution model";
+        else if (!(c->kappa >= 0.0) || !std::isfinite(c->kappa)) why = "kappa must be finite and >= 0";
+        else if (!(pi[0] > 0.0 && pi[1] > 0.0 && pi[2] > 0.0 && pi[3] > 0.0)) why = "F84/HKY85 need every pi > 0";
+        else if (cfg->incremental) why = "incremental rescoring supports F81 only";
+        if (why) {
+            c->err = why;
+            *out = c;
+            return MPCGS_E_ARG;
+        }
+        double Q[16];
+        rate_matrix(c->model, c->kappa, pi, Q);
+        eigen_system(Q, pi, gm);
+        u = 1.0;  // rates normalised to one substitution per unit time (S3); mu is not used
+    }
     // G0
     std::vector<int32_t> parent(c->nn);
     std::vector<double> age(c->nn);
@@ -735,7 +864,7 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
     c->L = L;
     c->Lpad = (L + 15) & ~15;
     c->incremental = cfg->incremental != 0;
-    Layout y = layout(n, Ls, c->Nmax, c->Mmax, c->precision, c->incremental);
+    Layout y = layout(n, Ls, c->Nmax, c->Mmax, c->precision, c->incremental, c->model);
     mpcgs_status st = MPCGS_OK;
     do {
         if (cudaStreamCreateWithFlags(&c->work, cudaStreamNonBlocking) != cudaSuccess ||
@@ -809,6 +938,9 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
         s.iee = (double*)(b + y.iee);
         s.cinfo = (int32_t*)(b + y.cinfo);
         s.gen_order = (int32_t*)(b + y.gen_order);
+        s.model = c->model ? 1 : 0;
+        s.gm = c->model ? (const double*)(b + y.gm) : nullptr;
+        s.sched_P = c->model ? (void*)(b + y.sched_P) : nullptr;
         s.Mmax = c->Mmax;
         c->theta_cnt = (unsigned*)(b + y.theta_cnt);
         c->score_out = (double*)(b + y.score_out);
@@ -826,6 +958,10 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
         if (cudaMemcpyAsync((void*)s.codes, padded.data(), padded.size(), cudaMemcpyHostToDevice, c->work) != cudaSuccess ||
             cudaMemcpyAsync(c->codes2, packed.data(), packed.size() * 4, cudaMemcpyHostToDevice, c->work) != cudaSuccess) {
             st = fail(c, MPCGS_E_CUDA, "codes upload");
+            break;
+        }
+        if (s.gm && cudaMemcpyAsync((void*)s.gm, gm, sizeof(gm), cudaMemcpyHostToDevice, c->work) != cudaSuccess) {
+            st = fail(c, MPCGS_E_CUDA, "model upload");
             break;
         }
         if (s.site_w &&

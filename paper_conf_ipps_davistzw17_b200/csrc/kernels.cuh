@@ -28,6 +28,8 @@ struct PruneArgs {
     double pi[4];
     const uint32_t* sched_op;  // [ntrees][nops]
     const void* sched_e;       // [ntrees][nops] float4 / double4
+    const double* gm;          // general model (f4): [36] eigen-system of Q, else nullptr (F81)
+    void* sched_P;             // general model: [ntrees][nops][32] P matrices (float / double)
     int tiles, sites_per_cta;
     const double* site_w;      // [L] pattern counts (compressed sites, f3) or nullptr
     const int32_t* tree_need;  // [ntrees] register need of each tree's schedule (nullable)
@@ -42,7 +44,7 @@ int prune_depth_for(int n);
 int prune_max_need(int n);
 int prune_need_cap(int n);
 int prune_batch_sites(int n, int precision);  // sites_per_cta must be a multiple of this
-bool prune_uses_tables(int n, int precision);
+bool prune_uses_tables(int n, int precision, bool general_model = false);
 cudaError_t launch_prune(const PruneArgs& a, int ntrees, int depth, int precision, cudaStream_t st,
                          int* n_launched = nullptr);
 

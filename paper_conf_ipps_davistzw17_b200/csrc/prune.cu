@@ -14,6 +14,7 @@
 // end (Eq. 22 read as a product over sites, S4).  CTA sums are reduced in a
 // fixed order by the last CTA of each tree (deterministic, P22).
 #include <algorithm>
+#include <type_traits>
 
 #include "arith.cuh"
 #include "common.cuh"
@@ -66,12 +67,98 @@ __device__ __forceinline__ void op_ss(T (&R)[D][4], const typename Traits<T>::E4
     }
 }
 
+// ---- general reversible model: per-op P matrices {P_a, P_b}
+// (row-major, row = parent state) formed by k_pmat; the tip vector of state x is
+// column x of P (Eq. 19 with a one-hot child partial), a branch is P . R.
+template <typename T>
+__device__ __forceinline__ void gm_tip(T (&v)[4], const T* __restrict__ P, int x) {
+#pragma unroll
+    for (int i = 0; i < 4; ++i) v[i] = __ldg(P + i * 4 + x);
+}
+
+template <typename T>
+__device__ __forceinline__ void gm_branch(T (&R)[4], const T* __restrict__ P) {
+    T o[4];
+#pragma unroll
+    for (int i = 0; i < 4; ++i) {
+        T v = P[i * 4] * R[0];
+        v = fma(P[i * 4 + 1], R[1], v);
+        v = fma(P[i * 4 + 2], R[2], v);
+        o[i] = fma(P[i * 4 + 3], R[3], v);
+    }
+#pragma unroll
+    for (int i = 0; i < 4; ++i) R[i] = o[i];
+}
+
+template <typename T, int D, int S>
+__device__ __forceinline__ void gm_tt(T (&R)[D][4], uint32_t code, const T* __restrict__ P,
+                                      const uint8_t* __restrict__ codes, int Lpad, int site, int& scale) {
+    if constexpr (S < D) {
+        int ta = (code >> 6) & 2047, tb = (code >> 17) & 2047;
+        T va[4], vb[4];
+        gm_tip<T>(va, P, __ldg(codes + (size_t)ta * Lpad + site));
+        gm_tip<T>(vb, P + 16, __ldg(codes + (size_t)tb * Lpad + site));
+#pragma unroll
+        for (int i = 0; i < 4; ++i) R[S][i] = va[i] * vb[i];
+        maybe_rescale(R[S], scale);
+    }
+}
+
+template <typename T, int D, int S>
+__device__ __forceinline__ void gm_ts(T (&R)[D][4], uint32_t code, const T* __restrict__ P,
+                                      const uint8_t* __restrict__ codes, int Lpad, int site, int& scale) {
+    if constexpr (S >= 1 && S <= D) {
+        int ta = (code >> 6) & 2047;
+        T va[4];
+        gm_tip<T>(va, P, __ldg(codes + (size_t)ta * Lpad + site));
+        gm_branch<T>(R[S - 1], P + 16);
+#pragma unroll
+        for (int i = 0; i < 4; ++i) R[S - 1][i] *= va[i];
+        maybe_rescale(R[S - 1], scale);
+    }
+}
+
+template <typename T, int D, int S>
+__device__ __forceinline__ void gm_ss(T (&R)[D][4], const T* __restrict__ P, int& scale) {
+    if constexpr (S >= 2 && S <= D) {
+        gm_branch<T>(R[S - 2], P);
+        gm_branch<T>(R[S - 1], P + 16);
+#pragma unroll
+        for (int i = 0; i < 4; ++i) R[S - 2][i] *= R[S - 1][i];
+        maybe_rescale(R[S - 2], scale);
+    }
+}
+
+#define MPCGS_GMCASE(S)                                                                       \
+    case (OP_TT | ((S) << 2)): gm_tt<T, D, S>(R, code, P, codes, Lpad, site, scale); break; \
+    case (OP_TS | ((S) << 2)): gm_ts<T, D, S>(R, code, P, codes, Lpad, site, scale); break; \
+    case (OP_SS | ((S) << 2)): gm_ss<T, D, S>(R, P, scale); break;
+
+// P matrices of every op's two children from the branch lengths in sched_e
+// ({t_a, 0, t_b, 0} under the general model): one thread per (tree, op, child).
+template <typename T>
+__global__ void __launch_bounds__(128) k_pmat(const void* sched_e, const double* gm, T* sched_P, int nops,
+                                              int ntrees) {
+    __shared__ double sgm[36];
+    if (threadIdx.x < 36) sgm[threadIdx.x] = gm[threadIdx.x];
+    __syncthreads();
+    const int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x;  // (tree * nops + op) * 2 + child
+    if (i >= (int64_t)ntrees * nops * 2) return;
+    const T* e = reinterpret_cast<const T*>(sched_e) + (i >> 1) * 4;
+    const double t = (double)e[(i & 1) ? 2 : 0];
+    double P[16];
+    pmat(sgm, t, P);
+    T* out = sched_P + i * 16;
+#pragma unroll
+    for (int k = 0; k < 16; ++k) out[k] = (T)P[k];
+}
+
 #define MPCGS_OPCASE(S)                                                                     \
     case (OP_TT | ((S) << 2)): op_tt<T, D, S>(R, code, ed, codes, Lpad, site, pi, scale); break; \
     case (OP_TS | ((S) << 2)): op_ts<T, D, S>(R, code, ed, codes, Lpad, site, pi, scale); break; \
     case (OP_SS | ((S) << 2)): op_ss<T, D, S>(R, ed, pi, scale); break;
 
-template <typename T, int D, bool W>
+template <typename T, int D, bool W, bool GM>
 __global__ void __launch_bounds__(PRUNE_THREADS) k_prune(PruneArgs a) {
     using E4 = typename Traits<T>::E4;
     extern __shared__ __align__(16) unsigned char smem_raw[];
@@ -87,9 +174,10 @@ __global__ void __launch_bounds__(PRUNE_THREADS) k_prune(PruneArgs a) {
     const E4* __restrict__ ge = reinterpret_cast<const E4*>(a.sched_e) + (size_t)tree * a.nops;
     for (int i = threadIdx.x; i < a.nops; i += blockDim.x) {
         s_op[i] = gop[i];
-        s_e[i] = ge[i];
+        if constexpr (!GM) s_e[i] = ge[i];
     }
     __syncthreads();
+    const T* __restrict__ gP = reinterpret_cast<const T*>(a.sched_P) + (size_t)tree * a.nops * 32;
 
     const T pi[4] = {(T)a.pi[0], (T)a.pi[1], (T)a.pi[2], (T)a.pi[3]};
     const uint8_t* __restrict__ codes = a.codes;
@@ -108,12 +196,22 @@ __global__ void __launch_bounds__(PRUNE_THREADS) k_prune(PruneArgs a) {
         int scale = 0;
         for (int op = 0; op < a.nops; ++op) {
             const uint32_t code = s_op[op];
-            const E4 ed = s_e[op];
-            switch (code & 63u) {
-                MPCGS_OPCASE(0) MPCGS_OPCASE(1) MPCGS_OPCASE(2) MPCGS_OPCASE(3) MPCGS_OPCASE(4)
-                MPCGS_OPCASE(5) MPCGS_OPCASE(6) MPCGS_OPCASE(7) MPCGS_OPCASE(8) MPCGS_OPCASE(9)
-                MPCGS_OPCASE(10) MPCGS_OPCASE(11)
-                default: break;
+            if constexpr (GM) {
+                const T* __restrict__ P = gP + (size_t)op * 32;
+                switch (code & 63u) {
+                    MPCGS_GMCASE(0) MPCGS_GMCASE(1) MPCGS_GMCASE(2) MPCGS_GMCASE(3) MPCGS_GMCASE(4)
+                    MPCGS_GMCASE(5) MPCGS_GMCASE(6) MPCGS_GMCASE(7) MPCGS_GMCASE(8) MPCGS_GMCASE(9)
+                    MPCGS_GMCASE(10) MPCGS_GMCASE(11)
+                    default: break;
+                }
+            } else {
+                const E4 ed = s_e[op];
+                switch (code & 63u) {
+                    MPCGS_OPCASE(0) MPCGS_OPCASE(1) MPCGS_OPCASE(2) MPCGS_OPCASE(3) MPCGS_OPCASE(4)
+                    MPCGS_OPCASE(5) MPCGS_OPCASE(6) MPCGS_OPCASE(7) MPCGS_OPCASE(8) MPCGS_OPCASE(9)
+                    MPCGS_OPCASE(10) MPCGS_OPCASE(11)
+                    default: break;
+                }
             }
         }
         // Eq. 21: L_s = sum_X pi_X L_root(X), root partial in R[0]
@@ -279,9 +377,21 @@ __device__ __forceinline__ void tab_tt(Stack<T, DR, SI>& st, uint32_t code, uint
     }
 }
 
-template <typename T, int DR, int SI, int S, int DMX>
+// branch data of an op: F81 {e_a, em_a, e_b, em_b}; general model (f4) a pointer
+// to the op's {P_a, P_b} in shared memory
+template <typename T, bool GM>
+using BranchData = std::conditional_t<GM, const T*, typename Traits<T>::E4>;
+
+template <typename T, bool GM, bool SECOND>
+__device__ __forceinline__ void branch_op(T (&v)[4], const BranchData<T, GM>& bd, const T (&pi)[4]) {
+    if constexpr (GM) gm_branch<T>(v, bd + (SECOND ? 16 : 0));
+    else if constexpr (SECOND) branch<T>(v, bd.z, bd.w, pi);
+    else branch<T>(v, bd.x, bd.y, pi);
+}
+
+template <typename T, int DR, int SI, int S, int DMX, bool GM>
 __device__ __forceinline__ void tab_ts(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff,
-                                       const typename Traits<T>::E4& ed, const T* s_tab, const Codes<SI>& c,
+                                       const BranchData<T, GM>& ed, const T* s_tab, const Codes<SI>& c,
                                        const T (&pi)[4], int (&scale)[SI]) {
     if constexpr (S >= 1 && S <= DMX) {
         constexpr int EB = 4 * sizeof(T);
@@ -293,7 +403,7 @@ __device__ __forceinline__ void tab_ts(Stack<T, DR, SI>& st, uint32_t code, uint
             T tip[4];
             ld4<T>(tip, reinterpret_cast<const T*>(base + c.template off<EB>(wa, k)));
             st.template get<S - 1>(k, v[k]);
-            branch<T>(v[k], ed.z, ed.w, pi);
+            branch_op<T, GM, true>(v[k], ed, pi);
 #pragma unroll
             for (int i = 0; i < 4; ++i) v[k][i] *= tip[i];
         }
@@ -303,8 +413,8 @@ __device__ __forceinline__ void tab_ts(Stack<T, DR, SI>& st, uint32_t code, uint
     }
 }
 
-template <typename T, int DR, int SI, int S, int DMX>
-__device__ __forceinline__ void tab_ss(Stack<T, DR, SI>& st, const typename Traits<T>::E4& ed, const T (&pi)[4],
+template <typename T, int DR, int SI, int S, int DMX, bool GM>
+__device__ __forceinline__ void tab_ss(Stack<T, DR, SI>& st, const BranchData<T, GM>& ed, const T (&pi)[4],
                                        int (&scale)[SI]) {
     if constexpr (S >= 2 && S <= DMX) {
         T v[SI][4];
@@ -313,8 +423,8 @@ __device__ __forceinline__ void tab_ss(Stack<T, DR, SI>& st, const typename Trai
             T w[4];
             st.template get<S - 2>(k, v[k]);
             st.template get<S - 1>(k, w);
-            branch<T>(v[k], ed.x, ed.y, pi);
-            branch<T>(w, ed.z, ed.w, pi);
+            branch_op<T, GM, false>(v[k], ed, pi);
+            branch_op<T, GM, true>(w, ed, pi);
 #pragma unroll
             for (int i = 0; i < 4; ++i) v[k][i] *= w[i];
         }
@@ -326,17 +436,17 @@ __device__ __forceinline__ void tab_ss(Stack<T, DR, SI>& st, const typename Trai
 
 #define MPCGS_TABCASE(S)                                                                          \
     case 3 * (S) + 0: tab_tt<T, DR, SI, PT, S, DMX>(st, code, toff, s_tab, cc, scale); break;       \
-    case 3 * (S) + 1: tab_ts<T, DR, SI, S, DMX>(st, code, toff, ed, s_tab, cc, pi, scale); break;     \
-    case 3 * (S) + 2: tab_ss<T, DR, SI, S, DMX>(st, ed, pi, scale); break;
+    case 3 * (S) + 1: tab_ts<T, DR, SI, S, DMX, GM>(st, code, toff, ed, s_tab, cc, pi, scale); break; \
+    case 3 * (S) + 2: tab_ss<T, DR, SI, S, DMX, GM>(st, ed, pi, scale); break;
 #define MPCGS_CASES_4 MPCGS_TABCASE(0) MPCGS_TABCASE(1) MPCGS_TABCASE(2) MPCGS_TABCASE(3) MPCGS_TABCASE(4)
 #define MPCGS_CASES_6 MPCGS_CASES_4 MPCGS_TABCASE(5) MPCGS_TABCASE(6)
 #define MPCGS_CASES_8 MPCGS_CASES_6 MPCGS_TABCASE(7) MPCGS_TABCASE(8)
 #define MPCGS_CASES_10 MPCGS_CASES_8 MPCGS_TABCASE(9) MPCGS_TABCASE(10)
 
 // one op for SI sites; the switch only has the (sp, type) labels a DMX-level tree can use
-template <typename T, int DR, int SI, bool PT, int DMX>
+template <typename T, int DR, int SI, bool PT, int DMX, bool GM>
 __device__ __forceinline__ void run_op(int di, Stack<T, DR, SI>& st, uint32_t code, uint32_t toff,
-                                       const typename Traits<T>::E4& ed, const T* s_tab, const Codes<SI>& cc,
+                                       const BranchData<T, GM>& ed, const T* s_tab, const Codes<SI>& cc,
                                        const T (&pi)[4], int (&scale)[SI]) {
     if constexpr (DMX <= 4) {
         switch (di) { MPCGS_CASES_4 default: __builtin_unreachable(); }
@@ -353,11 +463,11 @@ __host__ __device__ constexpr size_t align16(size_t x) { return (x + 15) & ~(siz
 
 // shared memory of the table kernel for trees of n tips whose register need is
 // at most `need` (spill levels above DR)
-template <typename T, int DR, int SI, bool PT>
+template <typename T, int DR, int SI, bool PT, bool GM = false>
 __host__ __device__ size_t tab_smem_bytes(int nops, int need) {
     const int n = nops + 1;
     const int spill = need > DR ? need - DR : 0;
-    return align16(sizeof(typename Traits<T>::E4) * nops) + align16(sizeof(T) * (PT ? 32 : 16) * (size_t)n) +
+    return align16((GM ? 32 * sizeof(T) : sizeof(typename Traits<T>::E4)) * nops) + align16(sizeof(T) * (PT ? 32 : 16) * (size_t)n) +
            align16(sizeof(uint2) * nops) + 2 * align16(Codes<SI>::buf_bytes(n)) +
            sizeof(T) * (size_t)spill * SI * 4 * PRUNE_THREADS;
 }
@@ -367,16 +477,18 @@ __host__ __device__ size_t tab_smem_bytes(int nops, int need) {
 #else
 #define MPCGS_TAB_BOUNDS __launch_bounds__(PRUNE_THREADS)
 #endif
-template <typename T, int DR, int SI, bool PT, int DMX, bool W>
+template <typename T, int DR, int SI, bool PT, int DMX, bool W, bool GM>
 __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
     using E4 = typename Traits<T>::E4;
     using CD = Codes<SI>;
     constexpr uint32_t TABE = PT ? 32u : 16u;  // table entries per tip
     constexpr int BATCH = CD::BATCH;  // sites per batch
+    constexpr size_t OPB = GM ? 32 * sizeof(T) : sizeof(E4);  // branch data bytes per op
     extern __shared__ __align__(16) unsigned char smem_raw[];
     const int nops = a.nops, n = nops + 1;
-    E4* s_e = reinterpret_cast<E4*>(smem_raw);
-    T* s_tab = reinterpret_cast<T*>(smem_raw + align16(sizeof(E4) * nops));
+    E4* s_e = reinterpret_cast<E4*>(smem_raw);  // F81: {e_a, em_a, e_b, em_b} per op
+    T* s_P = reinterpret_cast<T*>(smem_raw);    // general model: {P_a, P_b} per op
+    T* s_tab = reinterpret_cast<T*>(smem_raw + align16(OPB * nops));
     uint2* s_op = reinterpret_cast<uint2*>(reinterpret_cast<unsigned char*>(s_tab) + align16(sizeof(T) * TABE * n));
     unsigned char* s_cod = reinterpret_cast<unsigned char*>(s_op) + align16(sizeof(uint2) * nops);
     const size_t bufb = align16(CD::buf_bytes(n));
@@ -410,7 +522,11 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
     const E4* __restrict__ ge = reinterpret_cast<const E4*>(a.sched_e) + (size_t)tree * nops;
     for (int i = tid; i < nops; i += PRUNE_THREADS) {
         s_op[i].x = gop[i];
-        s_e[i] = ge[i];
+        if constexpr (!GM) s_e[i] = ge[i];
+    }
+    if constexpr (GM) {
+        const T* __restrict__ gP = reinterpret_cast<const T*>(a.sched_P) + (size_t)tree * nops * 32;
+        for (int i = tid; i < nops * 32; i += PRUNE_THREADS) s_P[i] = gP[i];
     }
     __syncthreads();
     if (tid < 32) {
@@ -438,6 +554,21 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
         const int op = idx >> 6, j = idx & 63;
         const uint32_t ty = s_op[op].x & 3u;
         T* tab = reinterpret_cast<T*>(reinterpret_cast<char*>(s_tab) + s_op[op].y);
+        if constexpr (GM) {  // entries are columns of P_a / P_b (row X = parent state)
+            const T* Pa = s_P + op * 32;
+            const T* Pb = Pa + 16;
+            if (ty == OP_TT && PT) {
+                const int xa = j >> 4, xb = (j >> 2) & 3, X = j & 3;
+                tab[j] = Pa[X * 4 + xa] * Pb[X * 4 + xb];
+            } else if (ty == OP_TT && j < 32) {
+                const int x = (j >> 2) & 3, X = j & 3;
+                tab[j] = j < 16 ? Pa[X * 4 + x] : Pb[X * 4 + x];
+            } else if (ty == OP_TS && j < 16) {
+                const int x = j >> 2, X = j & 3;
+                tab[j] = Pa[X * 4 + x];
+            }
+            continue;
+        }
         const E4 ed = s_e[op];
         if (ty == OP_TT && PT) {
             // cherry: entry (xa, xb) = P_{.,xa}(t_a) (.) P_{.,xb}(t_b)   (Eq. 19-20 at two tips)
@@ -494,9 +625,11 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
         for (int k = 0; k < SI; ++k) scale[k] = 0;
         for (int op = 0; op < nops; ++op) {
             const uint2 ox = s_op[op];
-            const E4 ed = s_e[op];
+            BranchData<T, GM> ed;
+            if constexpr (GM) ed = s_P + op * 32;
+            else ed = s_e[op];
             const int di = (int)((ox.x >> 2) & 15u) * 3 + (int)(ox.x & 3u);  // dense (sp, type) index
-            run_op<T, DR, SI, PT, DMX>(di, st, ox.x, ox.y, ed, s_tab, cc, pi, scale);
+            run_op<T, DR, SI, PT, DMX, GM>(di, st, ox.x, ox.y, ed, s_tab, cc, pi, scale);
         }
         const int site0 = s_begin + b * BATCH + tid * SI;
 #pragma unroll
@@ -536,10 +669,10 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
     }
 }
 
-template <typename T, int D, bool W>
+template <typename T, int D, bool W, bool GM>
 static cudaError_t launch_flat_w(const PruneArgs& a, int ntrees, cudaStream_t st) {
     size_t smem = (size_t)a.nops * (sizeof(typename Traits<T>::E4) + sizeof(uint32_t));
-    auto kern = k_prune<T, D, W>;
+    auto kern = k_prune<T, D, W, GM>;
     static size_t attr_bytes = 48 * 1024;  // raised once, outside graph capture (first launch is at init)
     if (smem > attr_bytes) {
         cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
@@ -553,13 +686,17 @@ static cudaError_t launch_flat_w(const PruneArgs& a, int ntrees, cudaStream_t st
 
 template <typename T, int D>
 static cudaError_t launch_flat(const PruneArgs& a, int ntrees, cudaStream_t st) {
-    return a.site_w ? launch_flat_w<T, D, true>(a, ntrees, st) : launch_flat_w<T, D, false>(a, ntrees, st);
+    if (a.gm)
+        return a.site_w ? launch_flat_w<T, D, true, true>(a, ntrees, st)
+                        : launch_flat_w<T, D, false, true>(a, ntrees, st);
+    return a.site_w ? launch_flat_w<T, D, true, false>(a, ntrees, st)
+                    : launch_flat_w<T, D, false, false>(a, ntrees, st);
 }
 
-template <typename T, int DR, int SI, bool PT, int DMX, bool W>
+template <typename T, int DR, int SI, bool PT, int DMX, bool W, bool GM>
 static cudaError_t launch_tab_w(const PruneArgs& a, int ntrees, cudaStream_t st) {
-    const size_t smem = tab_smem_bytes<T, DR, SI, PT>(a.nops, a.need_cap);
-    auto kern = k_prune_tab<T, DR, SI, PT, DMX, W>;
+    const size_t smem = tab_smem_bytes<T, DR, SI, PT, GM>(a.nops, a.need_cap);
+    auto kern = k_prune_tab<T, DR, SI, PT, DMX, W, GM>;
     static size_t attr_bytes = 48 * 1024;
     if (smem > attr_bytes) {
         cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
@@ -573,8 +710,11 @@ static cudaError_t launch_tab_w(const PruneArgs& a, int ntrees, cudaStream_t st)
 
 template <typename T, int DR, int SI, bool PT, int DMX>
 static cudaError_t launch_tab(const PruneArgs& a, int ntrees, cudaStream_t st) {
-    return a.site_w ? launch_tab_w<T, DR, SI, PT, DMX, true>(a, ntrees, st)
-                    : launch_tab_w<T, DR, SI, PT, DMX, false>(a, ntrees, st);
+    if (a.gm)
+        return a.site_w ? launch_tab_w<T, DR, SI, PT, DMX, true, true>(a, ntrees, st)
+                        : launch_tab_w<T, DR, SI, PT, DMX, false, true>(a, ntrees, st);
+    return a.site_w ? launch_tab_w<T, DR, SI, PT, DMX, true, false>(a, ntrees, st)
+                    : launch_tab_w<T, DR, SI, PT, DMX, false, false>(a, ntrees, st);
 }
 
 int prune_depth_for(int n) {
@@ -608,16 +748,18 @@ int prune_need_cap(int n) { return std::min(prune_max_need(n), PRUNE_DR + PRUNE_
 static bool product_tables(int n) { return n <= 128; }
 constexpr int PRUNE_SI_LARGE = 2;
 
-bool prune_uses_tables(int n, int precision) {
+template <typename T, bool GM>
+static size_t tab_bytes_for(int n) {
     const int cap = prune_need_cap(n);
-    const bool pt = product_tables(n);
+    constexpr int SI = sizeof(T) == 4 ? PRUNE_SI32 : PRUNE_SI64;
+    return product_tables(n) ? tab_smem_bytes<T, PRUNE_DR, SI, true, GM>(n - 1, cap)
+                             : tab_smem_bytes<T, PRUNE_DR, PRUNE_SI_LARGE, false, GM>(n - 1, cap);
+}
+
+bool prune_uses_tables(int n, int precision, bool general_model) {
     size_t bytes;
-    if (precision == 32)
-        bytes = pt ? tab_smem_bytes<float, PRUNE_DR, PRUNE_SI32, true>(n - 1, cap)
-                   : tab_smem_bytes<float, PRUNE_DR, PRUNE_SI_LARGE, false>(n - 1, cap);
-    else
-        bytes = pt ? tab_smem_bytes<double, PRUNE_DR, PRUNE_SI64, true>(n - 1, cap)
-                   : tab_smem_bytes<double, PRUNE_DR, PRUNE_SI_LARGE, false>(n - 1, cap);
+    if (precision == 32) bytes = general_model ? tab_bytes_for<float, true>(n) : tab_bytes_for<float, false>(n);
+    else bytes = general_model ? tab_bytes_for<double, true>(n) : tab_bytes_for<double, false>(n);
     return bytes <= 160 * 1024;
 }
 
@@ -644,9 +786,18 @@ static cudaError_t launch_flat_depth(const PruneArgs& a, int ntrees, int depth, 
 template <typename T, int SI>
 static cudaError_t launch_typed(PruneArgs a, int ntrees, int depth, cudaStream_t st, int& nl) {
     const int n = a.nops + 1;
-    nl = 1;
-    if (a.codes2 == nullptr || !prune_uses_tables(n, sizeof(T) == 4 ? 32 : 64)) {
+    nl = 0;
+    if (a.gm) {  // general model (f4): the P matrices of this launch's trees first
+        const int64_t threads = (int64_t)ntrees * a.nops * 2;
+        k_pmat<T><<<(unsigned)((threads + 127) / 128), 128, 0, st>>>(a.sched_e, a.gm, reinterpret_cast<T*>(a.sched_P),
+                                                                     a.nops, ntrees);
+        cudaError_t e = cudaGetLastError();
+        if (e != cudaSuccess) return e;
+        nl = 1;
+    }
+    if (a.codes2 == nullptr || !prune_uses_tables(n, sizeof(T) == 4 ? 32 : 64, a.gm != nullptr)) {
         a.tree_need = nullptr;  // flat kernel for every tree
+        nl += 1;
         return launch_flat_depth<T>(a, ntrees, depth, st);
     }
     a.need_cap = prune_need_cap(n);
@@ -654,8 +805,9 @@ static cudaError_t launch_typed(PruneArgs a, int ntrees, int depth, cudaStream_t
     if (!deep) a.tree_need = nullptr;
     cudaError_t e = product_tables(n) ? launch_tab_dmx<T, SI, true>(a, ntrees, st)
                                       : launch_tab_dmx<T, PRUNE_SI_LARGE, false>(a, ntrees, st);
+    nl += 1;
     if (e != cudaSuccess || !deep) return e;
-    nl = 2;
+    nl += 1;
     return launch_flat_depth<T>(a, ntrees, depth, st);  // trees with need > cap only
 }
 

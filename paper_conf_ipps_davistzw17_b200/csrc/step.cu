@@ -567,23 +567,18 @@ __global__ void __launch_bounds__(32) k_propose(DevState s, uint64_t seed, int64
         for (int v = A; v >= 0; v = sPar[v]) sNeed[v] = su_need(sNeed[sL[v - n]], sNeed[sR[v - n]]);
         s.tree_need[local] = sNeed[root];
     } else if (lane == 1) {
-        sh_d[2] = exp(-u * (t1 - ax));
-        sh_d[3] = -expm1(-u * (t1 - ax));
+        branch_data(s.model, u, t1 - ax, sh_d[2], sh_d[3]);
     } else if (lane == 2) {
-        sh_d[4] = exp(-u * (t1 - ay));
-        sh_d[5] = -expm1(-u * (t1 - ay));
+        branch_data(s.model, u, t1 - ay, sh_d[4], sh_d[5]);
     } else if (lane == 3) {
-        sh_d[6] = exp(-u * (t2 - az));
-        sh_d[7] = -expm1(-u * (t2 - az));
+        branch_data(s.model, u, t2 - az, sh_d[6], sh_d[7]);
     }
     __shared__ double sh_e2[4];
     if (lane == 4) {
-        sh_e2[0] = exp(-u * (t2 - t1));
-        sh_e2[1] = -expm1(-u * (t2 - t1));
+        branch_data(s.model, u, t2 - t1, sh_e2[0], sh_e2[1]);
     } else if (lane == 5) {
         const double lp = rootcase ? 0.0 : tAn - t2;
-        sh_e2[2] = exp(-u * lp);
-        sh_e2[3] = -expm1(-u * lp);
+        branch_data(s.model, u, lp, sh_e2[2], sh_e2[3]);
     }
     // S_G of the proposal: merge of the sorted fixed ages with {t1, t2} (Eq. 18 via
     MPCGS_TP(4);
@@ -812,17 +807,12 @@ __global__ void __launch_bounds__(DRAW_THREADS) k_draw(DevState s, uint64_t seed
         s.parent[T] = Par;
         s.age[T] = t1;
         s.age[Par] = t2;
-        s.e[x] = exp(-u * (t1 - s.age[x]));
-        s.em[x] = -expm1(-u * (t1 - s.age[x]));
-        s.e[y] = exp(-u * (t1 - s.age[y]));
-        s.em[y] = -expm1(-u * (t1 - s.age[y]));
-        s.e[z] = exp(-u * (t2 - s.age[z]));
-        s.em[z] = -expm1(-u * (t2 - s.age[z]));
-        s.e[T] = exp(-u * (t2 - t1));
-        s.em[T] = -expm1(-u * (t2 - t1));
+        branch_data(s.model, u, t1 - s.age[x], s.e[x], s.em[x]);
+        branch_data(s.model, u, t1 - s.age[y], s.e[y], s.em[y]);
+        branch_data(s.model, u, t2 - s.age[z], s.e[z], s.em[z]);
+        branch_data(s.model, u, t2 - t1, s.e[T], s.em[T]);
         const double lp = A < 0 ? 0.0 : s.age[A] - t2;
-        s.e[Par] = exp(-u * lp);
-        s.em[Par] = -expm1(-u * lp);
+        branch_data(s.model, u, lp, s.e[Par], s.em[Par]);
         auto nd = [&](int v) { return v < n ? 0 : s.need[v]; };
         s.need[T] = su_need(nd(x), nd(y));
         s.need[Par] = su_need(nd(T), nd(z));

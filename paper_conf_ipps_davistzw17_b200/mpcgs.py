@@ -39,8 +39,11 @@ class mpcgs_config(ctypes.Structure):
         ("init_age", ctypes.c_void_p), ("rank", ctypes.c_int32), ("world", ctypes.c_int32),
         ("nccl_id", ctypes.c_void_p), ("stream", ctypes.c_void_p), ("workspace", ctypes.c_void_p),
         ("workspace_bytes", ctypes.c_size_t), ("incremental", ctypes.c_int32),
-        ("compress_patterns", ctypes.c_int32),
+        ("compress_patterns", ctypes.c_int32), ("model", ctypes.c_int32), ("kappa", ctypes.c_double),
     ]
+
+
+MODELS = {"F81": 0, "F84": 1, "HKY85": 2}  # MPCGS_MODEL_*
 
 
 _lib = None
@@ -52,6 +55,8 @@ _SIGS = {
     "mpcgs_config_default": (None, [_P]),
     "mpcgs_workspace_bytes": (_sz, [_i32, _i32, _i32, _i64, _i32]),
     "mpcgs_workspace_bytes_ex": (_sz, [_i32, _i32, _i32, _i64, _i32, _i32]),
+    "mpcgs_workspace_bytes_cfg": (_sz, [_i32, _i32, _P]),
+    "mpcgs_transition": (_i32, [_i32, _f64, _P, _f64, _f64, _P]),
     "mpcgs_init": (_i32, [_P, _P, _f64, _P]),
     "mpcgs_init_phylip": (_i32, [ctypes.c_char_p, _P, _f64, _P]),
     "mpcgs_sample": (_i32, [_P, _i32, _i64, _u64]),
@@ -184,6 +189,17 @@ def mpcgs_philox(ctr, key):
     return out
 
 
+def mpcgs_transition(model, kappa, pi, mu, t):
+    """P(t) as the kernels form it (host-only entry point); model name or MPCGS_MODEL_* code."""
+    m = MODELS[model] if isinstance(model, str) else int(model)
+    p = _f64a(pi)
+    out = np.zeros(16, np.float64)
+    st = lib().mpcgs_transition(m, float(kappa), _ptr(p), float(mu), float(t), _ptr(out))
+    if st:
+        raise MpcgsError(st, "transition")
+    return out.reshape(4, 4)
+
+
 def mpcgs_nccl_unique_id():
     buf = ctypes.create_string_buffer(128)
     st = lib().mpcgs_nccl_unique_id(buf)
@@ -199,7 +215,7 @@ class Context:
     def __init__(self, rows, theta0, *, precision=64, burnin_steps=0, max_proposals=1024,
                  max_samples=1 << 20, base_freq=None, mu=0.0, init_tree=None, rank=0, world=1,
                  nccl_id=None, stream=None, workspace=None, phylip=None, incremental=False,
-                 compress_patterns=False):
+                 compress_patterns=False, model="F81", kappa=0.0):
         L = lib()
         cfg = mpcgs_config()
         L.mpcgs_config_default(ctypes.byref(cfg))
@@ -213,6 +229,8 @@ class Context:
         cfg.max_samples = int(max_samples)
         cfg.incremental = int(bool(incremental))
         cfg.compress_patterns = int(bool(compress_patterns))
+        cfg.model = MODELS[model] if isinstance(model, str) else int(model)
+        cfg.kappa = float(kappa)
         self._keep = []
         if init_tree is not None:
             p = _i32a(init_tree[0])

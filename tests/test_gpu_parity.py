@@ -52,6 +52,48 @@ def test_score_trees_matches_oracle(P, orc, precision, n, L):
         assert abs(g - want) <= LL_TOL[precision] * abs(want), (g, want)
 
 
+@pytest.mark.parametrize("model,kappa", [("F84", 2.0), ("HKY85", 6.0), ("F84", 0.0)])
+@pytest.mark.parametrize("precision", [64, 32])
+@pytest.mark.parametrize("n,L", [(3, 1), (12, 1000), (24, 129), (64, 1000), (256, 2000)])
+def test_score_trees_general_model(P, orc, model, kappa, precision, n, L):
+    """pruning under F84 / HKY85 (per-op P matrices from the
+    eigen-system, flat kernel) against the oracle's closed-form likelihood."""
+    rng = np.random.default_rng(11 * n + L)
+    pi = np.array([0.22, 0.28, 0.31, 0.19])
+    true_p, true_a = synth.coalescent_tree(n, 0.05, rng)
+    codes = synth.f81_alignment(true_p, true_a, L, pi, orc.default_rate(pi), rng)
+    trees = [synth.coalescent_tree(n, th, rng) for th in (0.01, 0.05, 0.3, 3.0)]
+    trees += [synth.shaped_tree(n, s, rng, scale=0.02) for s in ("caterpillar", "balanced")]
+    ctx = _ctx(P, codes, 0.05, tree=trees[0], precision=precision, base_freq=pi, max_proposals=8,
+               max_samples=16, model=model, kappa=kappa)
+    got = ctx.mpcgs_score_trees(np.stack([t[0] for t in trees]), np.stack([t[1] for t in trees]))
+    for (p, a), g in zip(trees, got):
+        want = orc.log_likelihood_model(model, kappa, codes, p, a, pi)
+        assert abs(g - want) <= LL_TOL[precision] * abs(want), (g, want)
+
+
+@pytest.mark.parametrize("model,kappa,name,N,steps", [("F84", 2.0, "c1", 16, 25), ("HKY85", 4.0, "c2", 32, 8),
+                                                      ("F84", 5.0, "c3", 64, 3)])
+def test_lockstep_general_model(P, orc, model, kappa, name, N, steps):
+    wl = synth.workload(name, L=400) if name != "c1" else synth.workload(name)
+    assert _lockstep(P, orc, wl, N, steps, wl["chain_seed"], model=model, kappa=kappa) <= max(2, steps // 4)
+
+
+def test_lockstep_general_model_compressed_fp32(P, orc):
+    wl = synth.workload("c1")
+    _lockstep(P, orc, wl, 16, 10, wl["chain_seed"], precision=32, compress=True, model="HKY85", kappa=3.0)
+
+
+def test_general_model_argument_errors(P):
+    rows = ["ACGT", "ACGA", "ACGG"]
+    with pytest.raises(P.MpcgsError):
+        P.Context(rows, 0.1, model="F84", kappa=2.0, incremental=True, max_proposals=4, max_samples=4)
+    with pytest.raises(P.MpcgsError):
+        P.Context(["AAGG", "AAGG", "GGAA"], 0.1, model="HKY85", kappa=2.0, max_proposals=4, max_samples=4)
+    with pytest.raises(P.MpcgsError):
+        P.Context(rows, 0.1, model=5, max_proposals=4, max_samples=4)
+
+
 def test_score_adversarial_branch_lengths(P, orc):
     rng = np.random.default_rng(3)
     n, L = 16, 300
@@ -95,15 +137,19 @@ def test_underflow_rescaling_long_alignment_many_tips(P, orc):
 
 
 # ------------------------------------------------------------------ GMH step (lock-step, P20)
-def _lockstep(P, orc, wl, N, steps, seed, K=None, precision=64, incremental=False, compress=False):
+def _lockstep(P, orc, wl, N, steps, seed, K=None, precision=64, incremental=False, compress=False,
+              model="F81", kappa=0.0):
     codes = wl["codes"]
     pi = orc.base_freqs(codes)
     u = orc.default_rate(pi)
     theta0 = wl["theta0"]
     parent, age = orc.upgma(codes, theta0)
-    gl = orc.log_likelihood(codes, parent, age, pi, u)
+    if model == "F81":
+        gl = orc.log_likelihood(codes, parent, age, pi, u)
+    else:
+        gl = orc.log_likelihood_model(model, kappa, codes, parent, age, pi)
     ctx = _ctx(P, codes, theta0, tree=(parent, age), precision=precision, max_proposals=N, max_samples=16,
-               incremental=incremental, compress_patterns=compress)
+               incremental=incremental, compress_patterns=compress, model=model, kappa=kappa)
     K = N if K is None else K
     height = age.max()
     skipped = 0
@@ -112,7 +158,7 @@ def _lockstep(P, orc, wl, N, steps, seed, K=None, precision=64, incremental=Fals
         gp, ga, g_ll, g_S = ctx.mpcgs_get_state()
         assert abs(g_ll - gl) <= LL_TOL[precision] * abs(gl)
         tr = ctx.mpcgs_step_trace(s, N, K, seed)
-        ref = orc.gmh_step(codes, pi, u, theta0, N, K, seed, s, parent, age, gl)
+        ref = orc.gmh_step(codes, pi, u, theta0, N, K, seed, s, parent, age, gl, model=model, kappa=kappa)
         assert tr["target"] == ref["target"]
         ok = ~ref["slot_flag"]
         ok[0] = True

@@ -124,3 +124,42 @@ def test_schedule_register_need_bound():
         assert depth == k
     parent, age = synth.shaped_tree(200, "caterpillar", np.random.default_rng(0))
     assert P.mpcgs_tree_schedule(parent, age, 1.0)[2] == 1
+
+
+@pytest.mark.parametrize("model", ["F84", "HKY85"])
+def test_library_transition_matches_oracle_closed_forms(orc, model):
+    """the library forms P(t) from the eigen-system of the normalised
+    rate matrix (host.cu rate_matrix / eigen_system, device pmat); the oracle from
+    the published closed forms (oracle.c orc_transition_model).  Independent routes."""
+    rng = np.random.default_rng(7)
+    pis = [np.full(4, 0.25), np.array([0.1, 0.2, 0.3, 0.4])] + [rng.dirichlet(np.ones(4) * 2) for _ in range(4)]
+    for pi in pis:
+        for kappa in [0.0, 0.5, 2.0, 10.0, 40.0]:
+            for t in [0.0, 1e-9, 1e-4, 0.05, 0.7, 3.0, 50.0]:
+                got = P.mpcgs_transition(model, kappa, pi, 0.0, t)
+                ref = orc.transition_model(model, kappa, t, pi)
+                assert np.allclose(got, ref, rtol=0, atol=2e-14), (model, pi, kappa, t)
+                assert np.all(got >= 0.0)
+
+
+def test_library_transition_f81_and_errors(orc):
+    pi = np.array([0.1, 0.2, 0.3, 0.4])
+    u = orc.default_rate(pi)
+    for t in [0.0, 0.3, 4.0]:
+        assert np.allclose(P.mpcgs_transition("F81", 0.0, pi, u, t), orc.transition(t, u, pi), rtol=0, atol=1e-15)
+    with pytest.raises(P.MpcgsError):
+        P.mpcgs_transition("F84", -1.0, pi, 0.0, 1.0)
+    with pytest.raises(P.MpcgsError):
+        P.mpcgs_transition("HKY85", 2.0, [0.5, 0.5, 0.0, 0.0], 0.0, 1.0)
+    with pytest.raises(P.MpcgsError):
+        P.mpcgs_transition(7, 2.0, pi, 0.0, 1.0)
+
+
+def test_workspace_bytes_cfg_counts_model_buffers():
+    cfg = B.mpcgs_config()
+    P.lib().mpcgs_config_default(ctypes.byref(cfg))
+    cfg.max_proposals, cfg.max_samples = 64, 20000
+    f81 = P.lib().mpcgs_workspace_bytes_cfg(12, 1000, ctypes.byref(cfg))
+    assert f81 == P.mpcgs_workspace_bytes(12, 1000, 64, 20000, 64)
+    cfg.model = P.MODELS["F84"]
+    assert P.lib().mpcgs_workspace_bytes_cfg(12, 1000, ctypes.byref(cfg)) >= f81 + 64 * 11 * 32 * 8

@@ -152,3 +152,25 @@ def test_chain_bookkeeping(orc):
     assert list(res["step"][16:32]) == [6] * 16
     assert list(res["step"][32:]) == [7] * 8
     assert np.all((res["slot"] >= 0) & (res["slot"] <= 16))
+
+
+def test_gmh_step_model_reduces_to_f81(orc):
+    """f4: F84 with kappa = 0 and HKY85 with kappa = 1 are F81, so the
+    model step must reproduce the F81 step: same target, trees, weights and draws."""
+    wl = synth.workload("c1")
+    codes = wl["codes"]
+    pi = orc.base_freqs(codes)
+    u = orc.default_rate(pi)
+    parent, age = orc.upgma(codes, wl["theta0"])
+    gl = orc.log_likelihood(codes, parent, age, pi, u)
+    ref = orc.gmh_step(codes, pi, u, wl["theta0"], 8, 8, 11, 3, parent, age, gl)
+    for model, kappa in (("F84", 0.0), ("HKY85", 1.0)):
+        got = orc.gmh_step(codes, pi, 0.0, wl["theta0"], 8, 8, 11, 3, parent, age, gl, model=model, kappa=kappa)
+        assert got["target"] == ref["target"]
+        assert np.array_equal(got["t12"], ref["t12"]) and np.array_equal(got["pair"], ref["pair"])
+        assert np.allclose(got["logL"], ref["logL"], rtol=1e-12, atol=0)
+        assert np.array_equal(got["draws"], ref["draws"])
+    # a real transition bias changes the likelihoods but not the proposals (Alg. 1)
+    got = orc.gmh_step(codes, pi, 0.0, wl["theta0"], 8, 8, 11, 3, parent, age, gl, model="HKY85", kappa=8.0)
+    assert np.array_equal(got["t12"], ref["t12"])
+    assert np.all(np.abs(got["logL"][1:] - ref["logL"][1:]) > 1e-6)
