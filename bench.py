@@ -298,7 +298,7 @@ def main():
     roof = {"bound": "alu", "achieved": achieved, "peak": pk[args.precision], "unit": "TFLOP/s",
             "frac": achieved / pk[args.precision],
             "traffic": traffic_from_profiles(f"{args.workload}_fp{args.precision}" + (f"_{args.model}" if gm else "")),
-            "kernel": "k_prune (flat, general model) + k_pmat" if gm else "k_prune_tab",
+            "kernel": "k_prune_tab (general model) + k_pmat" if gm else "k_prune_tab",
             "prune_share_of_step": prune_ms / loop_ms,
             "peak_source": f"derived: 148 SM x {'64 FP64' if args.precision == 64 else '128 FP32'} FMA lanes x 2 x "
                            f"{mhz:.0f} MHz (MEASURED_PEAKS sm_max_mhz)",

@@ -5,8 +5,10 @@ the CUDA runtime statically and loads NCCL with dlopen only when world > 1.
 """
 from __future__ import annotations
 
+import concurrent.futures
 import glob
 import os
+import shutil
 import subprocess
 import sys
 
@@ -17,7 +19,7 @@ INCLUDE = os.path.join(ROOT, "include")
 LIB = os.path.join(PKG, "libmpcgs.so")
 
 NVCC_FLAGS = [
-    "-std=c++17", "-O3", "-lineinfo", "-Xcompiler", "-fPIC", "-shared",
+    "-std=c++17", "-O3", "-lineinfo", "-Xcompiler", "-fPIC",
     "-gencode", "arch=compute_100a,code=sm_100a",
     "--expt-relaxed-constexpr", "-Xptxas", "-v",
 ]
@@ -44,13 +46,32 @@ def build(force: bool = False, verbose: bool = False, out: str = LIB, defines=()
         return LIB
     nvcc = os.environ.get("NVCC", "nvcc")
     tmp = out + f".tmp{os.getpid()}"
-    cmd = [nvcc, *NVCC_FLAGS, *[f"-D{d}" for d in defines], "-I", INCLUDE, "-I", CSRC, "-o", tmp, *sources(), "-ldl"]
-    res = subprocess.run(cmd, capture_output=True, text=True)
+    objdir = tmp + ".o.d"
+    os.makedirs(objdir, exist_ok=True)
+    srcs = sources()
+    objs = [os.path.join(objdir, os.path.basename(src) + ".o") for src in srcs]
+    base = [nvcc, *NVCC_FLAGS, *[f"-D{d}" for d in defines], "-I", INCLUDE, "-I", CSRC]
+
+    def compile_one(src_obj):  # one translation unit per nvcc process, all in parallel
+        src, obj = src_obj
+        return subprocess.run([*base, "-c", "-o", obj, src], capture_output=True, text=True)
+
+    with concurrent.futures.ThreadPoolExecutor(max_workers=max(1, min(len(srcs), os.cpu_count() or 1))) as ex:
+        results = list(ex.map(compile_one, zip(srcs, objs)))
+    log = "".join(r.stdout + r.stderr for r in results)
+    if any(r.returncode != 0 for r in results):
+        sys.stderr.write(log)
+        shutil.rmtree(objdir, ignore_errors=True)
+        raise RuntimeError("nvcc failed building libmpcgs.so")
+    res = subprocess.run([nvcc, "-shared", "-Xcompiler", "-fPIC", "-o", tmp, *objs, "-ldl"], capture_output=True,
+                         text=True)
+    shutil.rmtree(objdir, ignore_errors=True)
     if res.returncode != 0:
         sys.stderr.write(res.stdout + res.stderr)
-        raise RuntimeError("nvcc failed building libmpcgs.so")
+        raise RuntimeError("nvcc failed linking libmpcgs.so")
+    res.stderr = log
     if verbose:
-        sys.stderr.write(res.stderr)
+        sys.stderr.write(log)
     if out == LIB:
         with open(os.path.join(PKG, "build_ptxas.log"), "w") as f:
             f.write(res.stderr)

@@ -1,721 +1,9 @@
-// prune.cu -- Felsenstein pruning data likelihood (Eq. 19-22) of many
-// genealogies over all sites, F81 closed form (Eq. 20), on the CUDA cores.
-//
-// Grid: (site tiles, trees).  One CTA = one tree x one tile of sites; each
-// thread owns sites tid, tid+blockDim, ... of the tile.  The tree's post-order
-// schedule (common.cuh) is staged in shared memory once per CTA and read as
-// warp-uniform broadcasts; the live partial likelihood vectors of a site sit in
-// a register stack R[D][4] addressed only with compile-time indices (the switch
-// below dispatches on the uniform (type, sp) code), so no partial ever touches
-// shared or global memory.  Underflow: after each node the vector is rescaled
-// by an exact power of two when its max drops below 2^-TS (S5), with one
-// integer exponent per site.  Per-site likelihoods (Eq. 21) are multiplied
-// into a mantissa/exponent accumulator, so each thread takes one log at the
-// end (Eq. 22 read as a product over sites, S4).  CTA sums are reduced in a
-// fixed order by the last CTA of each tree (deterministic, P22).
-#include <algorithm>
-#include <type_traits>
-
-#include "arith.cuh"
-#include "common.cuh"
-#include "kernels.cuh"
+// prune.cu -- host-side routing of the pruning launches (kernels and launch
+// templates in prune_kernels.cuh; one translation unit per precision x model:
+// prune_f64.cu, prune_f32.cu, prune_f64_gm.cu, prune_f32_gm.cu).
+#include "prune_kernels.cuh"
 
 namespace mpcgs {
-
-template <typename T, int D, int S>
-__device__ __forceinline__ void op_tt(T (&R)[D][4], uint32_t code, const typename Traits<T>::E4& ed,
-                                      const uint8_t* __restrict__ codes, int Lpad, int site,
-                                      const T (&pi)[4], int& scale) {
-    if constexpr (S < D) {
-        int ta = (code >> 6) & 2047, tb = (code >> 17) & 2047;
-        int xa = __ldg(codes + (size_t)ta * Lpad + site);
-        int xb = __ldg(codes + (size_t)tb * Lpad + site);
-        T va[4], vb[4];
-        tipvec<T>(va, xa, ed.x, ed.y, pi);
-        tipvec<T>(vb, xb, ed.z, ed.w, pi);
-#pragma unroll
-        for (int i = 0; i < 4; ++i) R[S][i] = va[i] * vb[i];
-        maybe_rescale(R[S], scale);
-    }
-}
-
-template <typename T, int D, int S>
-__device__ __forceinline__ void op_ts(T (&R)[D][4], uint32_t code, const typename Traits<T>::E4& ed,
-                                      const uint8_t* __restrict__ codes, int Lpad, int site,
-                                      const T (&pi)[4], int& scale) {
-    if constexpr (S >= 1 && S <= D) {
-        int ta = (code >> 6) & 2047;
-        int xa = __ldg(codes + (size_t)ta * Lpad + site);
-        T va[4];
-        tipvec<T>(va, xa, ed.x, ed.y, pi);
-        branch<T>(R[S - 1], ed.z, ed.w, pi);
-#pragma unroll
-        for (int i = 0; i < 4; ++i) R[S - 1][i] *= va[i];
-        maybe_rescale(R[S - 1], scale);
-    }
-}
-
-template <typename T, int D, int S>
-__device__ __forceinline__ void op_ss(T (&R)[D][4], const typename Traits<T>::E4& ed, const T (&pi)[4],
-                                      int& scale) {
-    if constexpr (S >= 2 && S <= D) {
-        branch<T>(R[S - 2], ed.x, ed.y, pi);
-        branch<T>(R[S - 1], ed.z, ed.w, pi);
-#pragma unroll
-        for (int i = 0; i < 4; ++i) R[S - 2][i] *= R[S - 1][i];
-        maybe_rescale(R[S - 2], scale);
-    }
-}
-
-// ---- general reversible model: per-op P matrices {P_a, P_b}
-// (row-major, row = parent state) formed by k_pmat; the tip vector of state x is
-// column x of P (Eq. 19 with a one-hot child partial), a branch is P . R.
-template <typename T>
-__device__ __forceinline__ void gm_tip(T (&v)[4], const T* __restrict__ P, int x) {
-#pragma unroll
-    for (int i = 0; i < 4; ++i) v[i] = __ldg(P + i * 4 + x);
-}
-
-template <typename T>
-__device__ __forceinline__ void gm_branch(T (&R)[4], const T* __restrict__ P) {
-    T o[4];
-#pragma unroll
-    for (int i = 0; i < 4; ++i) {
-        T v = P[i * 4] * R[0];
-        v = fma(P[i * 4 + 1], R[1], v);
-        v = fma(P[i * 4 + 2], R[2], v);
-        o[i] = fma(P[i * 4 + 3], R[3], v);
-    }
-#pragma unroll
-    for (int i = 0; i < 4; ++i) R[i] = o[i];
-}
-
-template <typename T, int D, int S>
-__device__ __forceinline__ void gm_tt(T (&R)[D][4], uint32_t code, const T* __restrict__ P,
-                                      const uint8_t* __restrict__ codes, int Lpad, int site, int& scale) {
-    if constexpr (S < D) {
-        int ta = (code >> 6) & 2047, tb = (code >> 17) & 2047;
-        T va[4], vb[4];
-        gm_tip<T>(va, P, __ldg(codes + (size_t)ta * Lpad + site));
-        gm_tip<T>(vb, P + 16, __ldg(codes + (size_t)tb * Lpad + site));
-#pragma unroll
-        for (int i = 0; i < 4; ++i) R[S][i] = va[i] * vb[i];
-        maybe_rescale(R[S], scale);
-    }
-}
-
-template <typename T, int D, int S>
-__device__ __forceinline__ void gm_ts(T (&R)[D][4], uint32_t code, const T* __restrict__ P,
-                                      const uint8_t* __restrict__ codes, int Lpad, int site, int& scale) {
-    if constexpr (S >= 1 && S <= D) {
-        int ta = (code >> 6) & 2047;
-        T va[4];
-        gm_tip<T>(va, P, __ldg(codes + (size_t)ta * Lpad + site));
-        gm_branch<T>(R[S - 1], P + 16);
-#pragma unroll
-        for (int i = 0; i < 4; ++i) R[S - 1][i] *= va[i];
-        maybe_rescale(R[S - 1], scale);
-    }
-}
-
-template <typename T, int D, int S>
-__device__ __forceinline__ void gm_ss(T (&R)[D][4], const T* __restrict__ P, int& scale) {
-    if constexpr (S >= 2 && S <= D) {
-        gm_branch<T>(R[S - 2], P);
-        gm_branch<T>(R[S - 1], P + 16);
-#pragma unroll
-        for (int i = 0; i < 4; ++i) R[S - 2][i] *= R[S - 1][i];
-        maybe_rescale(R[S - 2], scale);
-    }
-}
-
-#define MPCGS_GMCASE(S)                                                                       \
-    case (OP_TT | ((S) << 2)): gm_tt<T, D, S>(R, code, P, codes, Lpad, site, scale); break; \
-    case (OP_TS | ((S) << 2)): gm_ts<T, D, S>(R, code, P, codes, Lpad, site, scale); break; \
-    case (OP_SS | ((S) << 2)): gm_ss<T, D, S>(R, P, scale); break;
-
-// P matrices of every op's two children from the branch lengths in sched_e
-// ({t_a, 0, t_b, 0} under the general model): one thread per (tree, op, child).
-template <typename T>
-__global__ void __launch_bounds__(128) k_pmat(const void* sched_e, const double* gm, T* sched_P, int nops,
-                                              int ntrees) {
-    __shared__ double sgm[36];
-    if (threadIdx.x < 36) sgm[threadIdx.x] = gm[threadIdx.x];
-    __syncthreads();
-    const int64_t i = (int64_t)blockIdx.x * blockDim.x + threadIdx.x;  // (tree * nops + op) * 2 + child
-    if (i >= (int64_t)ntrees * nops * 2) return;
-    const T* e = reinterpret_cast<const T*>(sched_e) + (i >> 1) * 4;
-    const double t = (double)e[(i & 1) ? 2 : 0];
-    double P[16];
-    pmat(sgm, t, P);
-    T* out = sched_P + i * 16;
-#pragma unroll
-    for (int k = 0; k < 16; ++k) out[k] = (T)P[k];
-}
-
-#define MPCGS_OPCASE(S)                                                                     \
-    case (OP_TT | ((S) << 2)): op_tt<T, D, S>(R, code, ed, codes, Lpad, site, pi, scale); break; \
-    case (OP_TS | ((S) << 2)): op_ts<T, D, S>(R, code, ed, codes, Lpad, site, pi, scale); break; \
-    case (OP_SS | ((S) << 2)): op_ss<T, D, S>(R, ed, pi, scale); break;
-
-template <typename T, int D, bool W, bool GM>
-__global__ void __launch_bounds__(PRUNE_THREADS) k_prune(PruneArgs a) {
-    using E4 = typename Traits<T>::E4;
-    extern __shared__ __align__(16) unsigned char smem_raw[];
-    E4* s_e = reinterpret_cast<E4*>(smem_raw);
-    uint32_t* s_op = reinterpret_cast<uint32_t*>(smem_raw + sizeof(E4) * a.nops);
-    __shared__ double s_red[PRUNE_THREADS / 32];
-    __shared__ bool s_last;
-
-    const int tree = blockIdx.y;
-    const int tile = blockIdx.x;
-    if (a.tree_need && a.tree_need[tree] <= a.need_cap) return;  // scored by the table pass
-    const uint32_t* __restrict__ gop = a.sched_op + (size_t)tree * a.nops;
-    const E4* __restrict__ ge = reinterpret_cast<const E4*>(a.sched_e) + (size_t)tree * a.nops;
-    for (int i = threadIdx.x; i < a.nops; i += blockDim.x) {
-        s_op[i] = gop[i];
-        if constexpr (!GM) s_e[i] = ge[i];
-    }
-    __syncthreads();
-    const T* __restrict__ gP = reinterpret_cast<const T*>(a.sched_P) + (size_t)tree * a.nops * 32;
-
-    const T pi[4] = {(T)a.pi[0], (T)a.pi[1], (T)a.pi[2], (T)a.pi[3]};
-    const uint8_t* __restrict__ codes = a.codes;
-    const int Lpad = a.Lpad;
-    const int s_begin = tile * a.sites_per_cta;
-    const int s_end = min(a.L, s_begin + a.sites_per_cta);
-
-    SiteAcc<W> acc;
-    T R[D][4];
-#pragma unroll
-    for (int i = 0; i < D; ++i)
-#pragma unroll
-        for (int j = 0; j < 4; ++j) R[i][j] = T(0);
-
-    for (int site = s_begin + threadIdx.x; site < s_end; site += blockDim.x) {
-        int scale = 0;
-        for (int op = 0; op < a.nops; ++op) {
-            const uint32_t code = s_op[op];
-            if constexpr (GM) {
-                const T* __restrict__ P = gP + (size_t)op * 32;
-                switch (code & 63u) {
-                    MPCGS_GMCASE(0) MPCGS_GMCASE(1) MPCGS_GMCASE(2) MPCGS_GMCASE(3) MPCGS_GMCASE(4)
-                    MPCGS_GMCASE(5) MPCGS_GMCASE(6) MPCGS_GMCASE(7) MPCGS_GMCASE(8) MPCGS_GMCASE(9)
-                    MPCGS_GMCASE(10) MPCGS_GMCASE(11)
-                    default: break;
-                }
-            } else {
-                const E4 ed = s_e[op];
-                switch (code & 63u) {
-                    MPCGS_OPCASE(0) MPCGS_OPCASE(1) MPCGS_OPCASE(2) MPCGS_OPCASE(3) MPCGS_OPCASE(4)
-                    MPCGS_OPCASE(5) MPCGS_OPCASE(6) MPCGS_OPCASE(7) MPCGS_OPCASE(8) MPCGS_OPCASE(9)
-                    MPCGS_OPCASE(10) MPCGS_OPCASE(11)
-                    default: break;
-                }
-            }
-        }
-        // Eq. 21: L_s = sum_X pi_X L_root(X), root partial in R[0]
-        T ls = pi[0] * R[0][0];
-        ls = fma(pi[1], R[0][1], ls);
-        ls = fma(pi[2], R[0][2], ls);
-        ls = fma(pi[3], R[0][3], ls);
-        acc.add((double)ls, scale, a.site_w, site);
-    }
-    // ln of this thread's product; -inf if any site likelihood was 0 (S6)
-    double ll = acc.total();
-    if (s_begin + (int)threadIdx.x >= s_end) ll = 0.0;
-
-    // block reduction in a fixed order
-#pragma unroll
-    for (int off = 16; off > 0; off >>= 1) ll += __shfl_down_sync(0xffffffffu, ll, off);
-    if ((threadIdx.x & 31) == 0) s_red[threadIdx.x >> 5] = ll;
-    __syncthreads();
-    if (threadIdx.x == 0) {
-        double t = 0.0;
-        for (int w = 0; w < (int)(blockDim.x >> 5); ++w) t += s_red[w];
-        a.tile_part[(size_t)tree * a.tiles + tile] = t;
-        __threadfence();
-        unsigned prev = atomicAdd(a.tile_cnt + tree, 1u);
-        s_last = (prev == (unsigned)(a.tiles - 1));
-    }
-    __syncthreads();
-    if (s_last && threadIdx.x == 0) {
-        __threadfence();
-        double t = 0.0;
-        const volatile double* tp = a.tile_part + (size_t)tree * a.tiles;
-        for (int k = 0; k < a.tiles; ++k) t += tp[k];
-        a.out[(size_t)(a.out_first + tree) * a.out_stride] = t;
-        a.tile_cnt[tree] = 0u;
-    }
-}
-
-// ============================================================================
-// Table kernel (the production path).  Tip codes are staged per site batch in
-// shared memory (2-bit packed, cp.async double buffer); every tip child reads
-// its 4-vector P_{.,x}(t) from a per-op 4x4 table and every cherry (two tip
-// children) its product vector from a 16x4 table, both built in shared memory
-// at CTA start; SI sites per thread are interleaved so that one dispatch and one
-// read of the op serve SI register stacks.  The register stack holds DR levels;
-// deeper levels (rare: need > DR) live in shared memory, so one compiled kernel
-// scores every tree shape.
-// ============================================================================
-__device__ __forceinline__ void cp_async16(void* smem, const void* gmem) {
-    unsigned sa = (unsigned)__cvta_generic_to_shared(smem);
-    asm volatile("cp.async.cg.shared.global [%0], [%1], 16;\n" ::"r"(sa), "l"(gmem));
-}
-__device__ __forceinline__ void cp_async_commit() { asm volatile("cp.async.commit_group;\n" ::); }
-template <int N>
-__device__ __forceinline__ void cp_async_wait() { asm volatile("cp.async.wait_group %0;\n" ::"n"(N)); }
-
-template <typename T, int SI>
-__device__ __forceinline__ void rescale_sites(T (&v)[SI][4], int (&scale)[SI]) {
-    bool any = false;
-#pragma unroll
-    for (int q = 0; q < SI; ++q) any |= small4(v[q]);
-    if (__any_sync(0xffffffffu, any)) {
-#pragma unroll
-        for (int q = 0; q < SI; ++q) {
-            const int k = rescale_k(v[q]);
-            const T f = pow2(k, T(0));
-            v[q][0] *= f; v[q][1] *= f; v[q][2] *= f; v[q][3] *= f;
-            scale[q] += k;
-        }
-    }
-}
-
-// Register stack of DR levels per site, deeper levels in shared memory laid out
-// [level][site k][state X][thread] (conflict-free).
-template <typename T, int DR, int SI>
-struct Stack {
-    T r[SI][DR][4];
-    T* sm;  // this thread's column of the spill area
-    template <int S>
-    __device__ __forceinline__ void get(int k, T (&v)[4]) const {
-        if constexpr (S < DR) {
-            v[0] = r[k][S][0]; v[1] = r[k][S][1]; v[2] = r[k][S][2]; v[3] = r[k][S][3];
-        } else {
-#pragma unroll
-            for (int x = 0; x < 4; ++x) v[x] = sm[(((S - DR) * SI + k) * 4 + x) * PRUNE_THREADS];
-        }
-    }
-    template <int S>
-    __device__ __forceinline__ void put(int k, const T (&v)[4]) {
-        if constexpr (S < DR) {
-            r[k][S][0] = v[0]; r[k][S][1] = v[1]; r[k][S][2] = v[2]; r[k][S][3] = v[3];
-        } else {
-#pragma unroll
-            for (int x = 0; x < 4; ++x) sm[(((S - DR) * SI + k) * 4 + x) * PRUNE_THREADS] = v[x];
-        }
-    }
-};
-
-// Tip codes of the current site batch in shared memory, 2-bit packed (16 sites
-// per 32-bit word, a thread's SI sites adjacent).  The byte offset of a site's
-// table entry is one funnel rotation and one mask: rotating the word right by
-// (bit position - log2(entry bytes)) puts the 2-bit code at the entry-size bit.
-template <int SI>
-struct Codes {
-    const unsigned char* base;  // this batch's buffer
-    int wofs;                   // word index of this thread's sites
-    uint32_t rb[SI], ra[SI];    // rotations for the code * EB and code * 4 * EB offsets
-    static constexpr int BATCH = PRUNE_THREADS * SI;
-    static constexpr int WB = BATCH / 16;
-    template <int EB>
-    __device__ __forceinline__ void init(int tid) {
-        constexpr int LG = EB == 32 ? 5 : 4;
-        wofs = (tid * SI) >> 4;
-#pragma unroll
-        for (int k = 0; k < SI; ++k) {
-            const int p = ((tid * SI) & 15) * 2 + 2 * k;  // bit position of site k's code
-            rb[k] = (uint32_t)(p - LG) & 31u;
-            ra[k] = (uint32_t)(p - LG - 2) & 31u;
-        }
-    }
-    __device__ __forceinline__ uint32_t word(int tip) const {
-        return reinterpret_cast<const uint32_t*>(base)[tip * WB + wofs];
-    }
-    template <int EB>
-    __device__ __forceinline__ uint32_t off(uint32_t w, int k) const {  // code * EB
-        return __funnelshift_r(w, w, rb[k]) & (3u * EB);
-    }
-    template <int EB>
-    __device__ __forceinline__ uint32_t off4(uint32_t w, int k) const {  // code * 4 * EB
-        return __funnelshift_r(w, w, ra[k]) & (12u * EB);
-    }
-    static constexpr size_t buf_bytes(int n) { return (size_t)n * WB * 4; }
-};
-
-constexpr uint32_t TAB_CHECK = 0x80000000u;  // toff flag: the cherry table can hold small vectors
-
-template <typename T, int DR, int SI, bool PT, int S, int DMX>
-__device__ __forceinline__ void tab_tt(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, const T* s_tab,
-                                       const Codes<SI>& c, int (&scale)[SI]) {
-    if constexpr (S < DMX) {
-        constexpr int EB = 4 * sizeof(T);
-        const uint32_t wa = c.word((code >> 6) & 2047);
-        const uint32_t wb = c.word((code >> 17) & 2047);
-        const char* base = reinterpret_cast<const char*>(s_tab) + (toff & ~TAB_CHECK);
-        T v[SI][4];
-        if constexpr (PT) {  // 16x4 product table of the cherry
-#pragma unroll
-            for (int k = 0; k < SI; ++k)
-                ld4<T>(v[k], reinterpret_cast<const T*>(base + c.template off4<EB>(wa, k) + c.template off<EB>(wb, k)));
-            if (toff & TAB_CHECK) rescale_sites<T, SI>(v, scale);
-        } else {             // two 4x4 tip tables, multiplied here
-#pragma unroll
-            for (int k = 0; k < SI; ++k) {
-                T w[4];
-                ld4<T>(v[k], reinterpret_cast<const T*>(base + c.template off<EB>(wa, k)));
-                ld4<T>(w, reinterpret_cast<const T*>(base + 16 * sizeof(T) + c.template off<EB>(wb, k)));
-#pragma unroll
-                for (int i = 0; i < 4; ++i) v[k][i] *= w[i];
-            }
-            rescale_sites<T, SI>(v, scale);
-        }
-#pragma unroll
-        for (int k = 0; k < SI; ++k) st.template put<S>(k, v[k]);
-    }
-}
-
-// branch data of an op: F81 {e_a, em_a, e_b, em_b}; general model (f4) a pointer
-// to the op's {P_a, P_b} in shared memory
-template <typename T, bool GM>
-using BranchData = std::conditional_t<GM, const T*, typename Traits<T>::E4>;
-
-template <typename T, bool GM, bool SECOND>
-__device__ __forceinline__ void branch_op(T (&v)[4], const BranchData<T, GM>& bd, const T (&pi)[4]) {
-    if constexpr (GM) gm_branch<T>(v, bd + (SECOND ? 16 : 0));
-    else if constexpr (SECOND) branch<T>(v, bd.z, bd.w, pi);
-    else branch<T>(v, bd.x, bd.y, pi);
-}
-
-template <typename T, int DR, int SI, int S, int DMX, bool GM>
-__device__ __forceinline__ void tab_ts(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff,
-                                       const BranchData<T, GM>& ed, const T* s_tab, const Codes<SI>& c,
-                                       const T (&pi)[4], int (&scale)[SI]) {
-    if constexpr (S >= 1 && S <= DMX) {
-        constexpr int EB = 4 * sizeof(T);
-        const uint32_t wa = c.word((code >> 6) & 2047);
-        const char* base = reinterpret_cast<const char*>(s_tab) + toff;
-        T v[SI][4];
-#pragma unroll
-        for (int k = 0; k < SI; ++k) {
-            T tip[4];
-            ld4<T>(tip, reinterpret_cast<const T*>(base + c.template off<EB>(wa, k)));
-            st.template get<S - 1>(k, v[k]);
-            branch_op<T, GM, true>(v[k], ed, pi);
-#pragma unroll
-            for (int i = 0; i < 4; ++i) v[k][i] *= tip[i];
-        }
-        rescale_sites<T, SI>(v, scale);
-#pragma unroll
-        for (int k = 0; k < SI; ++k) st.template put<S - 1>(k, v[k]);
-    }
-}
-
-template <typename T, int DR, int SI, int S, int DMX, bool GM>
-__device__ __forceinline__ void tab_ss(Stack<T, DR, SI>& st, const BranchData<T, GM>& ed, const T (&pi)[4],
-                                       int (&scale)[SI]) {
-    if constexpr (S >= 2 && S <= DMX) {
-        T v[SI][4];
-#pragma unroll
-        for (int k = 0; k < SI; ++k) {
-            T w[4];
-            st.template get<S - 2>(k, v[k]);
-            st.template get<S - 1>(k, w);
-            branch_op<T, GM, false>(v[k], ed, pi);
-            branch_op<T, GM, true>(w, ed, pi);
-#pragma unroll
-            for (int i = 0; i < 4; ++i) v[k][i] *= w[i];
-        }
-        rescale_sites<T, SI>(v, scale);
-#pragma unroll
-        for (int k = 0; k < SI; ++k) st.template put<S - 2>(k, v[k]);
-    }
-}
-
-#define MPCGS_TABCASE(S)                                                                          \
-    case 3 * (S) + 0: tab_tt<T, DR, SI, PT, S, DMX>(st, code, toff, s_tab, cc, scale); break;       \
-    case 3 * (S) + 1: tab_ts<T, DR, SI, S, DMX, GM>(st, code, toff, ed, s_tab, cc, pi, scale); break; \
-    case 3 * (S) + 2: tab_ss<T, DR, SI, S, DMX, GM>(st, ed, pi, scale); break;
-#define MPCGS_CASES_4 MPCGS_TABCASE(0) MPCGS_TABCASE(1) MPCGS_TABCASE(2) MPCGS_TABCASE(3) MPCGS_TABCASE(4)
-#define MPCGS_CASES_6 MPCGS_CASES_4 MPCGS_TABCASE(5) MPCGS_TABCASE(6)
-#define MPCGS_CASES_8 MPCGS_CASES_6 MPCGS_TABCASE(7) MPCGS_TABCASE(8)
-#define MPCGS_CASES_10 MPCGS_CASES_8 MPCGS_TABCASE(9) MPCGS_TABCASE(10)
-
-// one op for SI sites; the switch only has the (sp, type) labels a DMX-level tree can use
-template <typename T, int DR, int SI, bool PT, int DMX, bool GM>
-__device__ __forceinline__ void run_op(int di, Stack<T, DR, SI>& st, uint32_t code, uint32_t toff,
-                                       const BranchData<T, GM>& ed, const T* s_tab, const Codes<SI>& cc,
-                                       const T (&pi)[4], int (&scale)[SI]) {
-    if constexpr (DMX <= 4) {
-        switch (di) { MPCGS_CASES_4 default: __builtin_unreachable(); }
-    } else if constexpr (DMX <= 6) {
-        switch (di) { MPCGS_CASES_6 default: __builtin_unreachable(); }
-    } else if constexpr (DMX <= 8) {
-        switch (di) { MPCGS_CASES_8 default: __builtin_unreachable(); }
-    } else {
-        switch (di) { MPCGS_CASES_10 default: __builtin_unreachable(); }
-    }
-}
-
-__host__ __device__ constexpr size_t align16(size_t x) { return (x + 15) & ~(size_t)15; }
-
-// shared memory of the table kernel for trees of n tips whose register need is
-// at most `need` (spill levels above DR)
-template <typename T, int DR, int SI, bool PT, bool GM = false>
-__host__ __device__ size_t tab_smem_bytes(int nops, int need) {
-    const int n = nops + 1;
-    const int spill = need > DR ? need - DR : 0;
-    return align16((GM ? 32 * sizeof(T) : sizeof(typename Traits<T>::E4)) * nops) + align16(sizeof(T) * (PT ? 32 : 16) * (size_t)n) +
-           align16(sizeof(uint2) * nops) + 2 * align16(Codes<SI>::buf_bytes(n)) +
-           sizeof(T) * (size_t)spill * SI * 4 * PRUNE_THREADS;
-}
-
-#ifdef MPCGS_MINB  // tuning builds only: min CTAs per SM (caps registers)
-#define MPCGS_TAB_BOUNDS __launch_bounds__(PRUNE_THREADS, MPCGS_MINB)
-#else
-#define MPCGS_TAB_BOUNDS __launch_bounds__(PRUNE_THREADS)
-#endif
-template <typename T, int DR, int SI, bool PT, int DMX, bool W, bool GM>
-__global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
-    using E4 = typename Traits<T>::E4;
-    using CD = Codes<SI>;
-    constexpr uint32_t TABE = PT ? 32u : 16u;  // table entries per tip
-    constexpr int BATCH = CD::BATCH;  // sites per batch
-    constexpr size_t OPB = GM ? 32 * sizeof(T) : sizeof(E4);  // branch data bytes per op
-    extern __shared__ __align__(16) unsigned char smem_raw[];
-    const int nops = a.nops, n = nops + 1;
-    E4* s_e = reinterpret_cast<E4*>(smem_raw);  // F81: {e_a, em_a, e_b, em_b} per op
-    T* s_P = reinterpret_cast<T*>(smem_raw);    // general model: {P_a, P_b} per op
-    T* s_tab = reinterpret_cast<T*>(smem_raw + align16(OPB * nops));
-    uint2* s_op = reinterpret_cast<uint2*>(reinterpret_cast<unsigned char*>(s_tab) + align16(sizeof(T) * TABE * n));
-    unsigned char* s_cod = reinterpret_cast<unsigned char*>(s_op) + align16(sizeof(uint2) * nops);
-    const size_t bufb = align16(CD::buf_bytes(n));
-    T* s_spill = reinterpret_cast<T*>(s_cod + 2 * bufb);
-    __shared__ double s_red[PRUNE_THREADS / 32];
-    __shared__ bool s_last;
-
-    const int tid = threadIdx.x;
-    const int tree = blockIdx.y;
-    const int tile = blockIdx.x;
-    const int s_begin = tile * a.sites_per_cta;
-    const int s_end = min(a.L, s_begin + a.sites_per_cta);
-    const int nb = (s_end - s_begin + BATCH - 1) / BATCH;
-    if (a.tree_need && a.tree_need[tree] > a.need_cap) return;  // deeper tree: scored by the flat pass
-
-    auto issue = [&](int b, int buf) {
-        const int site0 = s_begin + b * BATCH;
-        unsigned char* dst = s_cod + (size_t)buf * bufb;
-        constexpr int WB = CD::WB, CH = WB / 4;  // 16-byte chunks per tip row
-        const uint32_t* src = a.codes2 + (site0 >> 4);
-        for (int c = tid; c < n * CH; c += PRUNE_THREADS) {
-            const int tip = c / CH, q = c - tip * CH;
-            cp_async16(dst + ((size_t)tip * WB + q * 4) * 4, src + (size_t)tip * a.W2 + q * 4);
-        }
-        cp_async_commit();
-    };
-    if (nb > 0) issue(0, 0);
-
-    // schedule, then per-op table byte offsets (warp 0 scan), then the tables
-    const uint32_t* __restrict__ gop = a.sched_op + (size_t)tree * nops;
-    const E4* __restrict__ ge = reinterpret_cast<const E4*>(a.sched_e) + (size_t)tree * nops;
-    for (int i = tid; i < nops; i += PRUNE_THREADS) {
-        s_op[i].x = gop[i];
-        if constexpr (!GM) s_e[i] = ge[i];
-    }
-    if constexpr (GM) {
-        const T* __restrict__ gP = reinterpret_cast<const T*>(a.sched_P) + (size_t)tree * nops * 32;
-        for (int i = tid; i < nops * 32; i += PRUNE_THREADS) s_P[i] = gP[i];
-    }
-    __syncthreads();
-    if (tid < 32) {
-        uint32_t carry = 0;
-        for (int base = 0; base < nops; base += 32) {
-            const int i = base + tid;
-            uint32_t sz = 0;
-            if (i < nops) {
-                const uint32_t ty = s_op[i].x & 3u;
-                sz = ty == OP_TT ? 2u * TABE : (ty == OP_TS ? 16u : 0u);
-            }
-            uint32_t x = sz;
-#pragma unroll
-            for (int o = 1; o < 32; o <<= 1) {
-                const uint32_t y = __shfl_up_sync(0xffffffffu, x, o);
-                if (tid >= o) x += y;
-            }
-            if (i < nops) s_op[i].y = (carry + x - sz) * (uint32_t)sizeof(T);  // byte offset
-            carry += __shfl_sync(0xffffffffu, x, 31);
-        }
-    }
-    __syncthreads();
-    const T pi[4] = {(T)a.pi[0], (T)a.pi[1], (T)a.pi[2], (T)a.pi[3]};
-    for (int idx = tid; idx < nops * 64; idx += PRUNE_THREADS) {
-        const int op = idx >> 6, j = idx & 63;
-        const uint32_t ty = s_op[op].x & 3u;
-        T* tab = reinterpret_cast<T*>(reinterpret_cast<char*>(s_tab) + s_op[op].y);
-        if constexpr (GM) {  // entries are columns of P_a / P_b (row X = parent state)
-            const T* Pa = s_P + op * 32;
-            const T* Pb = Pa + 16;
-            if (ty == OP_TT && PT) {
-                const int xa = j >> 4, xb = (j >> 2) & 3, X = j & 3;
-                tab[j] = Pa[X * 4 + xa] * Pb[X * 4 + xb];
-            } else if (ty == OP_TT && j < 32) {
-                const int x = (j >> 2) & 3, X = j & 3;
-                tab[j] = j < 16 ? Pa[X * 4 + x] : Pb[X * 4 + x];
-            } else if (ty == OP_TS && j < 16) {
-                const int x = j >> 2, X = j & 3;
-                tab[j] = Pa[X * 4 + x];
-            }
-            continue;
-        }
-        const E4 ed = s_e[op];
-        if (ty == OP_TT && PT) {
-            // cherry: entry (xa, xb) = P_{.,xa}(t_a) (.) P_{.,xb}(t_b)   (Eq. 19-20 at two tips)
-            const int xa = j >> 4, xb = (j >> 2) & 3, X = j & 3;
-            const T va = (X == xa ? (T)ed.x : T(0)) + (T)ed.y * pick4(pi, xa);
-            const T vb = (X == xb ? (T)ed.z : T(0)) + (T)ed.w * pick4(pi, xb);
-            tab[j] = va * vb;
-        } else if (ty == OP_TT && j < 32) {  // two tip tables: a at [0, 16), b at [16, 32)
-            const int x = (j >> 2) & 3, X = j & 3;
-            tab[j] = j < 16 ? (X == x ? (T)ed.x : T(0)) + (T)ed.y * pick4(pi, x)
-                            : (X == x ? (T)ed.z : T(0)) + (T)ed.w * pick4(pi, x);
-        } else if (ty == OP_TS && j < 16) {
-            const int x = j >> 2, X = j & 3;
-            tab[j] = (X == x ? (T)ed.x : T(0)) + (T)ed.y * pick4(pi, x);
-        }
-    }
-    __syncthreads();
-    // flag cherry tables with an entry whose max is below the rescale threshold
-    for (int op = tid; op < nops && PT; op += PRUNE_THREADS) {
-        if ((s_op[op].x & 3u) != OP_TT) continue;
-        const T* tab = reinterpret_cast<const T*>(reinterpret_cast<const char*>(s_tab) + s_op[op].y);
-        bool small = false;
-        for (int e = 0; e < 16; ++e) {
-            T v[4];
-            ld4<T>(v, tab + 4 * e);
-            small |= small4(v);
-        }
-        if (small) s_op[op].y |= TAB_CHECK;
-    }
-
-    SiteAcc<W> acc;
-    Stack<T, DR, SI> st;
-    st.sm = s_spill + tid;
-#pragma unroll
-    for (int k = 0; k < SI; ++k)
-#pragma unroll
-        for (int i = 0; i < DR; ++i)
-#pragma unroll
-            for (int j = 0; j < 4; ++j) st.r[k][i][j] = T(0);
-
-    CD cc;
-    cc.template init<4 * sizeof(T)>(tid);
-    for (int b = 0; b < nb; ++b) {
-        if (b + 1 < nb) {
-            issue(b + 1, (b + 1) & 1);
-            cp_async_wait<1>();
-        } else {
-            cp_async_wait<0>();
-        }
-        __syncthreads();
-        cc.base = s_cod + (size_t)(b & 1) * bufb;
-        int scale[SI];
-#pragma unroll
-        for (int k = 0; k < SI; ++k) scale[k] = 0;
-        for (int op = 0; op < nops; ++op) {
-            const uint2 ox = s_op[op];
-            BranchData<T, GM> ed;
-            if constexpr (GM) ed = s_P + op * 32;
-            else ed = s_e[op];
-            const int di = (int)((ox.x >> 2) & 15u) * 3 + (int)(ox.x & 3u);  // dense (sp, type) index
-            run_op<T, DR, SI, PT, DMX, GM>(di, st, ox.x, ox.y, ed, s_tab, cc, pi, scale);
-        }
-        const int site0 = s_begin + b * BATCH + tid * SI;
-#pragma unroll
-        for (int k = 0; k < SI; ++k) {
-            T root[4];
-            st.template get<0>(k, root);
-            T ls = pi[0] * root[0];   // Eq. 21
-            ls = fma(pi[1], root[1], ls);
-            ls = fma(pi[2], root[2], ls);
-            ls = fma(pi[3], root[3], ls);
-            if (site0 + k < s_end) acc.add((double)ls, scale[k], a.site_w, site0 + k);  // padding not counted
-        }
-        __syncthreads();  // the buffer of batch b is refilled in iteration b+1
-    }
-    double ll = acc.total();
-
-#pragma unroll
-    for (int off = 16; off > 0; off >>= 1) ll += __shfl_down_sync(0xffffffffu, ll, off);
-    if ((tid & 31) == 0) s_red[tid >> 5] = ll;
-    __syncthreads();
-    if (tid == 0) {
-        double t = 0.0;
-        for (int w = 0; w < PRUNE_THREADS / 32; ++w) t += s_red[w];
-        a.tile_part[(size_t)tree * a.tiles + tile] = t;
-        __threadfence();
-        const unsigned prev = atomicAdd(a.tile_cnt + tree, 1u);
-        s_last = (prev == (unsigned)(a.tiles - 1));
-    }
-    __syncthreads();
-    if (s_last && tid == 0) {
-        __threadfence();
-        double t = 0.0;
-        const volatile double* tp = a.tile_part + (size_t)tree * a.tiles;
-        for (int k = 0; k < a.tiles; ++k) t += tp[k];
-        a.out[(size_t)(a.out_first + tree) * a.out_stride] = t;
-        a.tile_cnt[tree] = 0u;
-    }
-}
-
-template <typename T, int D, bool W, bool GM>
-static cudaError_t launch_flat_w(const PruneArgs& a, int ntrees, cudaStream_t st) {
-    size_t smem = (size_t)a.nops * (sizeof(typename Traits<T>::E4) + sizeof(uint32_t));
-    auto kern = k_prune<T, D, W, GM>;
-    static size_t attr_bytes = 48 * 1024;  // raised once, outside graph capture (first launch is at init)
-    if (smem > attr_bytes) {
-        cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-        if (e != cudaSuccess) return e;
-        attr_bytes = smem;
-    }
-    dim3 grid(a.tiles, ntrees);
-    kern<<<grid, PRUNE_THREADS, smem, st>>>(a);
-    return cudaGetLastError();
-}
-
-template <typename T, int D>
-static cudaError_t launch_flat(const PruneArgs& a, int ntrees, cudaStream_t st) {
-    if (a.gm)
-        return a.site_w ? launch_flat_w<T, D, true, true>(a, ntrees, st)
-                        : launch_flat_w<T, D, false, true>(a, ntrees, st);
-    return a.site_w ? launch_flat_w<T, D, true, false>(a, ntrees, st)
-                    : launch_flat_w<T, D, false, false>(a, ntrees, st);
-}
-
-template <typename T, int DR, int SI, bool PT, int DMX, bool W, bool GM>
-static cudaError_t launch_tab_w(const PruneArgs& a, int ntrees, cudaStream_t st) {
-    const size_t smem = tab_smem_bytes<T, DR, SI, PT, GM>(a.nops, a.need_cap);
-    auto kern = k_prune_tab<T, DR, SI, PT, DMX, W, GM>;
-    static size_t attr_bytes = 48 * 1024;
-    if (smem > attr_bytes) {
-        cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-        if (e != cudaSuccess) return e;
-        attr_bytes = smem;
-    }
-    dim3 grid(a.tiles, ntrees);
-    kern<<<grid, PRUNE_THREADS, smem, st>>>(a);
-    return cudaGetLastError();
-}
-
-template <typename T, int DR, int SI, bool PT, int DMX>
-static cudaError_t launch_tab(const PruneArgs& a, int ntrees, cudaStream_t st) {
-    if (a.gm)
-        return a.site_w ? launch_tab_w<T, DR, SI, PT, DMX, true, true>(a, ntrees, st)
-                        : launch_tab_w<T, DR, SI, PT, DMX, false, true>(a, ntrees, st);
-    return a.site_w ? launch_tab_w<T, DR, SI, PT, DMX, true, false>(a, ntrees, st)
-                    : launch_tab_w<T, DR, SI, PT, DMX, false, false>(a, ntrees, st);
-}
 
 int prune_depth_for(int n) {
     int d = 0;
@@ -732,7 +20,6 @@ int prune_max_need(int n) {
     return d < 1 ? 1 : d;
 }
 
-static bool product_tables(int n);
 // sites interleaved per thread: 4 for n <= 128 (product tables), 2 for larger
 // trees, whose codes / tables / spill levels take more shared memory
 static int prune_si(int n, int precision) {
@@ -745,8 +32,6 @@ int prune_batch_sites(int n, int precision) { return PRUNE_THREADS * prune_si(n,
 // deeper trees (rare) are scored by the flat kernel in a second pass
 int prune_need_cap(int n) { return std::min(prune_max_need(n), PRUNE_DR + PRUNE_SPILL); }
 
-static bool product_tables(int n) { return n <= 128; }
-constexpr int PRUNE_SI_LARGE = 2;
 
 template <typename T, bool GM>
 static size_t tab_bytes_for(int n) {
@@ -763,61 +48,15 @@ bool prune_uses_tables(int n, int precision, bool general_model) {
     return bytes <= 160 * 1024;
 }
 
-template <typename T, int SI, bool PT>
-static cudaError_t launch_tab_dmx(const PruneArgs& a, int ntrees, cudaStream_t st) {
-    switch (a.need_cap) {
-        case 1: case 2: case 3: case 4: return launch_tab<T, PRUNE_DR, SI, PT, 4>(a, ntrees, st);
-        case 5: case 6: return launch_tab<T, PRUNE_DR, SI, PT, 6>(a, ntrees, st);
-        case 7: case 8: return launch_tab<T, PRUNE_DR, SI, PT, 8>(a, ntrees, st);
-        default: return launch_tab<T, PRUNE_DR, SI, PT, 10>(a, ntrees, st);
-    }
-}
-
-template <typename T>
-static cudaError_t launch_flat_depth(const PruneArgs& a, int ntrees, int depth, cudaStream_t st) {
-    switch (depth) {
-        case 4: return launch_flat<T, 4>(a, ntrees, st);
-        case 6: return launch_flat<T, 6>(a, ntrees, st);
-        case 8: return launch_flat<T, 8>(a, ntrees, st);
-        default: return launch_flat<T, 10>(a, ntrees, st);
-    }
-}
-
-template <typename T, int SI>
-static cudaError_t launch_typed(PruneArgs a, int ntrees, int depth, cudaStream_t st, int& nl) {
-    const int n = a.nops + 1;
-    nl = 0;
-    if (a.gm) {  // general model (f4): the P matrices of this launch's trees first
-        const int64_t threads = (int64_t)ntrees * a.nops * 2;
-        k_pmat<T><<<(unsigned)((threads + 127) / 128), 128, 0, st>>>(a.sched_e, a.gm, reinterpret_cast<T*>(a.sched_P),
-                                                                     a.nops, ntrees);
-        cudaError_t e = cudaGetLastError();
-        if (e != cudaSuccess) return e;
-        nl = 1;
-    }
-    if (a.codes2 == nullptr || !prune_uses_tables(n, sizeof(T) == 4 ? 32 : 64, a.gm != nullptr)) {
-        a.tree_need = nullptr;  // flat kernel for every tree
-        nl += 1;
-        return launch_flat_depth<T>(a, ntrees, depth, st);
-    }
-    a.need_cap = prune_need_cap(n);
-    const bool deep = prune_max_need(n) > a.need_cap && a.tree_need != nullptr;
-    if (!deep) a.tree_need = nullptr;
-    cudaError_t e = product_tables(n) ? launch_tab_dmx<T, SI, true>(a, ntrees, st)
-                                      : launch_tab_dmx<T, PRUNE_SI_LARGE, false>(a, ntrees, st);
-    nl += 1;
-    if (e != cudaSuccess || !deep) return e;
-    nl += 1;
-    return launch_flat_depth<T>(a, ntrees, depth, st);  // trees with need > cap only
-}
-
 cudaError_t launch_prune(const PruneArgs& a, int ntrees, int depth, int precision, cudaStream_t st,
                          int* n_launched) {
     int nl = 0;
     cudaError_t e = cudaSuccess;
     if (ntrees > 0)
-        e = precision == 32 ? launch_typed<float, PRUNE_SI32>(a, ntrees, depth, st, nl)
-                            : launch_typed<double, PRUNE_SI64>(a, ntrees, depth, st, nl);
+        e = precision == 32 ? (a.gm ? launch_prune_typed<float, true>(a, ntrees, depth, st, nl)
+                                    : launch_prune_typed<float, false>(a, ntrees, depth, st, nl))
+                            : (a.gm ? launch_prune_typed<double, true>(a, ntrees, depth, st, nl)
+                                    : launch_prune_typed<double, false>(a, ntrees, depth, st, nl));
     if (n_launched) *n_launched = nl;
     return e;
 }

@@ -1,0 +1,6 @@
+// prune_f64_gm.cu -- instantiates the pruning kernels for FP64 partials, general reversible model (F84 / HKY85).
+#include "prune_kernels.cuh"
+
+namespace mpcgs {
+template cudaError_t launch_prune_typed<double, true>(PruneArgs, int, int, cudaStream_t, int&);
+}  // namespace mpcgs
