@@ -90,8 +90,14 @@ void orc_base_freqs(int n, int L, const uint8_t* codes, double pi[4]) {
     double count[4] = {0.0, 0.0, 0.0, 0.0};
     long i, total = (long)n * (long)L;
     int X;
-    for (i = 0; i < total; ++i) count[codes[i]] += 1.0;
-    for (X = 0; X < 4; ++X) pi[X] = total > 0 ? count[X] / (double)total : 0.25;
+    double known = 0.0;
+    /* ambiguity codes (>= 16, S24) are not counted */
+    for (i = 0; i < total; ++i)
+        if (codes[i] < 4) {
+            count[codes[i]] += 1.0;
+            known += 1.0;
+        }
+    for (X = 0; X < 4; ++X) pi[X] = known > 0 ? count[X] / known : 0.25;
 }
 
 /* u = 1 / (1 - sum pi^2) so that branch lengths are expected substitutions (S3). */
@@ -249,9 +255,12 @@ static void prune_node(prune_work* w, int v, int site) {
     double* out = w->lnL + 4 * v;
     int X, Y, side;
     if (v < w->n) {
-        /* Tips are indicator vectors (L673-676): L = 1 for the observed base. */
+        /* Tips are indicator vectors (L673-676): L = 1 for the observed base; an
+           ambiguity code (16 + set, reading S24) is the indicator
+           of its set of bases (Felsenstein 1981, 2004 ch. 16). */
         int code = w->codes[(long)v * w->L + site];
-        for (X = 0; X < 4; ++X) out[X] = (X == code) ? 0.0 : -INFINITY;
+        int set = code < 4 ? 1 << code : code - 16;
+        for (X = 0; X < 4; ++X) out[X] = ((set >> X) & 1) ? 0.0 : -INFINITY;
         return;
     }
     for (X = 0; X < 4; ++X) out[X] = 0.0;
@@ -1063,7 +1072,11 @@ int orc_upgma(int n, int L, const uint8_t* codes, double theta0, int32_t* parent
         alive[i] = 1;
         for (j = 0; j < n; ++j) {
             int diff = 0;
-            for (s = 0; s < L; ++s) diff += codes[(long)i * L + s] != codes[(long)j * L + s];
+            for (s = 0; s < L; ++s) {   /* a difference: disjoint base sets (S24) */
+                int a = codes[(long)i * L + s], b = codes[(long)j * L + s];
+                int sa = a < 4 ? 1 << a : a - 16, sb = b < 4 ? 1 << b : b - 16;
+                diff += (sa & sb) == 0;
+            }
             D[i * nn + j] = (double)diff;
         }
     }

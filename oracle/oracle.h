@@ -16,7 +16,9 @@
  * interior nodes n..2n-2; parent[root] = -1; age[] in coalescent time units
  * (mutation units, S22).  Children of a node are ordered by ascending id.
  *
- * Tip data: codes[tip*L + site] in {0,1,2,3} = {A,C,G,T}.
+ * Tip data: codes[tip*L + site] in {0,1,2,3} = {A,C,G,T}, or 16 + m for an
+ * ambiguity code whose base set is the 4-bit mask m (bit X = base X; 16 + 15 = N;
+ * SURVEY 8(f) f4, reading S24).
  */
 #ifndef MPCGS_ORACLE_H
 #define MPCGS_ORACLE_H

@@ -115,8 +115,32 @@ def random_alignment(n: int, L: int, rng: np.random.Generator, pi=None):
     return rng.choice(4, size=(n, L), p=pi).astype(np.uint8)
 
 
+# IUPAC ambiguity letters by base-set mask (bit X = base X of A, C, G, T); code 16 + mask
+IUPAC = {1: "A", 2: "C", 4: "G", 8: "T", 5: "R", 10: "Y", 6: "S", 9: "W", 12: "K", 3: "M",
+         14: "B", 13: "D", 11: "H", 7: "V", 15: "N"}
+
+
+def _letter(c: int) -> str:
+    return BASES[c] if c < 4 else IUPAC[c - 16]
+
+
 def to_strings(codes):
-    return ["".join(BASES[c] for c in row) for row in np.asarray(codes)]
+    return ["".join(_letter(int(c)) for c in row) for row in np.asarray(codes)]
+
+
+def ambiguate(codes, frac: float, rng: np.random.Generator, gap_frac: float = 0.0):
+    """Replace a fraction of characters by ambiguity codes (16 + mask, the mask
+    drawn uniformly among the multi-base IUPAC sets containing the replaced base,
+    N included) and a further fraction by N (gaps / missing data)."""
+    out = np.array(codes, dtype=np.uint8, copy=True)
+    multi = [m for m in IUPAC if bin(m).count("1") > 1]
+    having = [np.array([m for m in multi if (m >> x) & 1], dtype=np.uint8) for x in range(4)]
+    hit = np.argwhere(rng.random(out.shape) < frac)
+    for i, j in hit:  # a set that contains the base it replaces
+        out[i, j] = 16 + rng.choice(having[int(codes[i][j]) if codes[i][j] < 4 else 0])
+    gap = rng.random(out.shape) < gap_frac
+    out[gap] = 16 + 15
+    return out
 
 
 # BASELINE.json configs: (n, L, N, M, theta0)

@@ -245,3 +245,78 @@ def test_model_pruning_equals_brute_force(orc, model):
         total += prob
     assert np.isclose(orc.log_likelihood_model(model, kappa, codes, parent, age, pi), np.log(total).sum(),
                       rtol=1e-12)
+
+
+# ------------------------------------------------------------------ ambiguity codes (f4, reading S24)
+def _set_of(code):
+    return [code] if code < 4 else [x for x in range(4) if ((code - 16) >> x) & 1]
+
+
+@pytest.mark.parametrize("model", ["F81", "HKY85"])
+def test_ambiguity_pruning_equals_brute_force(orc, model):
+    """An ambiguous tip's likelihood is the sum over the bases it stands for:
+    brute force over interior assignments AND tip resolutions."""
+    rng = np.random.default_rng(91)
+    n, kappa = 4, 2.5
+    parent, age = synth.shaped_tree(n, "random", rng, scale=0.3)
+    pi = np.array([0.3, 0.2, 0.15, 0.35])
+    u = orc.default_rate(pi)
+    codes = synth.ambiguate(synth.random_alignment(n, 20, rng, pi), 0.3, rng, gap_frac=0.1)
+    assert (codes >= 16).any() and (codes == 31).any()
+    Q = _f81_Q(pi, u) if model == "F81" else _model_Q(model, kappa, pi)
+    nn = 2 * n - 1
+    root = int(np.where(parent < 0)[0][0])
+    Pb = {v: scipy.linalg.expm(Q * (age[parent[v]] - age[v])) for v in range(nn) if parent[v] >= 0}
+    interior = list(range(n, nn))
+    want = np.zeros(codes.shape[1])
+    for s in range(codes.shape[1]):
+        tot = 0.0
+        for assign in itertools.product(range(4), repeat=len(interior)):
+            st = dict(zip(interior, assign))
+            prob = pi[st[root]]
+            for v in range(nn):
+                if parent[v] < 0:
+                    continue
+                if v < n:
+                    prob *= sum(Pb[v][st[parent[v]], x] for x in _set_of(int(codes[v, s])))
+                else:
+                    prob *= Pb[v][st[parent[v]], st[v]]
+            tot += prob
+        want[s] = np.log(tot)
+    if model == "F81":
+        got = orc.log_likelihood(codes, parent, age, pi, u)
+    else:
+        got = orc.log_likelihood_model(model, kappa, codes, parent, age, pi)
+    assert np.isclose(got, want.sum(), rtol=1e-12)
+
+
+def test_ambiguity_special_cases(orc):
+    rng = np.random.default_rng(5)
+    n = 6
+    parent, age = synth.coalescent_tree(n, 0.5, rng)
+    pi = np.array([0.1, 0.2, 0.3, 0.4])
+    u = orc.default_rate(pi)
+    codes = synth.random_alignment(n, 12, rng, pi)
+    # an all-N column has site likelihood exactly 1
+    c2 = codes.copy()
+    c2[:, 3] = 31
+    _, site = orc.log_likelihood(c2, parent, age, pi, u, site_ll=True)
+    assert site[3] == 0.0 or abs(site[3]) < 1e-15
+    # a one-base "set" is that base
+    c3 = codes.copy()
+    c3[2, :] = 16 + (1 << codes[2, :])
+    assert orc.log_likelihood(c3, parent, age, pi, u) == orc.log_likelihood(codes, parent, age, pi, u)
+    # R at a tip = A there + G there (linearity of Eq. 19 in a tip vector)
+    cA, cG, cR = codes.copy(), codes.copy(), codes.copy()
+    cA[1, 5], cG[1, 5], cR[1, 5] = 0, 2, 16 + 5
+    sA = orc.log_likelihood(cA, parent, age, pi, u, site_ll=True)[1][5]
+    sG = orc.log_likelihood(cG, parent, age, pi, u, site_ll=True)[1][5]
+    sR = orc.log_likelihood(cR, parent, age, pi, u, site_ll=True)[1][5]
+    assert np.isclose(np.exp(sR), np.exp(sA) + np.exp(sG), rtol=1e-13)
+    # base frequencies ignore ambiguous characters; UPGMA: N differs from nothing
+    amb = synth.ambiguate(codes, 0.5, rng)
+    known = amb[amb < 4]
+    assert np.allclose(orc.base_freqs(amb), np.bincount(known, minlength=4) / known.size)
+    two = np.array([[0, 1, 2, 3], [31, 31, 31, 31], [0, 1, 2, 0]], np.uint8)
+    p, a = orc.upgma(two, 1.0)
+    assert a[p[1]] <= 1e-6 + 1e-12  # row 1 joins first (distance 0 to everything)
