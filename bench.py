@@ -189,7 +189,9 @@ def workload_config(args, wl):
                         "per proposal and site" if getattr(args, "incremental", False) else "full pruning (5.2.2)")
             + ("; compressed site patterns (f3): partials/s counts all L columns" if getattr(args, "compress", False)
                else ""),
-            "model": args.model + ("" if args.model == "F81" else f" (kappa {args.kappa}; SURVEY 8(f) f4)")}
+            "model": args.model + ("" if args.model == "F81" else f" (kappa {args.kappa}; SURVEY 8(f) f4)"),
+            "ambiguity": (f"{args.ambiguity:g} of characters IUPAC ambiguity codes + {args.ambiguity / 2:g} N "
+                          "(SURVEY 8(f) f4; flat kernel)" if args.ambiguity > 0 else "none")}
 
 
 def main():
@@ -215,6 +217,9 @@ def main():
     ap.add_argument("--model", default="F81", choices=["F81", "F84", "HKY85"],
                     help="substitution model (F84 / HKY85: SURVEY 8(f) f4)")
     ap.add_argument("--kappa", type=float, default=2.0, help="F84 / HKY85 transition/transversion parameter")
+    ap.add_argument("--ambiguity", type=float, default=0.0,
+                    help="fraction of characters replaced by IUPAC ambiguity codes (plus half that as N); "
+                         "SURVEY 8(f) f4")
     args = ap.parse_args()
     args.warmup = max(args.warmup, 3)
 
@@ -229,6 +234,11 @@ def main():
     if args.N:
         over["N"] = args.N
     wl = synth.workload(args.workload, theta_true=args.theta_true, **over)
+    if args.ambiguity > 0:  # IUPAC ambiguity codes + gaps (reading S24)
+        import numpy as np
+
+        wl["codes"] = synth.ambiguate(wl["codes"], args.ambiguity, np.random.default_rng(wl["chain_seed"] + 7),
+                                      gap_frac=args.ambiguity / 2)
     if args.impl == "reference":
         run_reference(args, wl, rank)
         return
@@ -270,7 +280,7 @@ def main():
     ctx = P.Context(rows, wl["theta0"], precision=args.precision, max_proposals=N, max_samples=N * total_steps,
                     init_tree=(wl["true_parent"], wl["true_age"]), rank=rank, world=world, nccl_id=nccl_id,
                     stream=stream, incremental=args.incremental, compress_patterns=args.compress,
-                    model=args.model, kappa=args.kappa)
+                    model=args.model, kappa=args.kappa, ambiguity=args.ambiguity > 0)
     # warm-up (untimed): W steps
     ctx.mpcgs_sample(N, N * args.warmup, wl["chain_seed"])
     ctx.mpcgs_set_timing(3)   # per-step + per-prune CUDA events, L2 flush between steps
@@ -298,7 +308,8 @@ def main():
     roof = {"bound": "alu", "achieved": achieved, "peak": pk[args.precision], "unit": "TFLOP/s",
             "frac": achieved / pk[args.precision],
             "traffic": traffic_from_profiles(f"{args.workload}_fp{args.precision}" + (f"_{args.model}" if gm else "")),
-            "kernel": "k_prune_tab (general model) + k_pmat" if gm else "k_prune_tab",
+            "kernel": ("k_prune (flat, base-set tips)" if args.ambiguity > 0 else "k_prune_tab")
+                      + (" + general model (F84/HKY85)" if gm else ""),
             "prune_share_of_step": prune_ms / loop_ms,
             "peak_source": f"derived: 148 SM x {'64 FP64' if args.precision == 64 else '128 FP32'} FMA lanes x 2 x "
                            f"{mhz:.0f} MHz (MEASURED_PEAKS sm_max_mhz)",
@@ -314,7 +325,8 @@ def main():
         ctx2 = P.Context(rows, wl["theta0"], precision=args.precision, max_proposals=N, max_samples=N * args.steps,
                          init_tree=(wl["true_parent"], wl["true_age"]), rank=rank, world=world,
                          nccl_id=fresh_nccl_id(), stream=stream, incremental=args.incremental,
-                         compress_patterns=args.compress, model=args.model, kappa=args.kappa)
+                         compress_patterns=args.compress, model=args.model, kappa=args.kappa,
+                         ambiguity=args.ambiguity > 0)
         ctx2.mpcgs_sample(N, N * args.steps, wl["chain_seed"] + 1)
         smp = ctx2.mpcgs_get_samples()
         barrier()
@@ -336,7 +348,8 @@ def main():
     if not args.incremental and not args.no_incremental_block and not gm:
         ctx3 = P.Context(rows, wl["theta0"], precision=args.precision, max_proposals=N,
                          max_samples=N * (args.warmup + args.steps), init_tree=(wl["true_parent"], wl["true_age"]),
-                         rank=rank, world=world, nccl_id=fresh_nccl_id(), stream=stream, incremental=True)
+                         rank=rank, world=world, nccl_id=fresh_nccl_id(), stream=stream, incremental=True,
+                         ambiguity=args.ambiguity > 0)
         ctx3.mpcgs_sample(N, N * args.warmup, wl["chain_seed"])
         ctx3.mpcgs_set_timing(3)
         barrier()

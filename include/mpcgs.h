@@ -99,6 +99,12 @@ typedef struct {
                               one expected substitution per unit time (mu is ignored), every
                               pi > 0, incremental = 0 (else MPCGS_E_ARG) */
     double kappa;          /* transition/transversion parameter of F84 / HKY85 (>= 0) */
+    int32_t ambiguity;     /* 1: accept IUPAC ambiguity codes (M R W S Y K V H D B N, '-' and '?'
+                              as N; either case) as the set of bases they stand for (SURVEY 8(f)
+                              f4, reading S24: the tip's partial vector is the set's indicator;
+                              empirical pi counts A/C/G/T only; UPGMA counts a site as a
+                              difference when the two sets are disjoint).  0: S2, anything but
+                              ACGT -> MPCGS_E_ALIGNMENT */
 } mpcgs_config;
 
 #define MPCGS_MODEL_F81 0
@@ -228,7 +234,8 @@ void mpcgs_free(mpcgs_ctx* ctx);
 /* [host-only] Proposal slots owned by `rank`: slots first..first+count-1 of 1..N. */
 mpcgs_status mpcgs_shard_range(int32_t n_proposals, int32_t rank, int32_t world, int32_t* first,
                                int32_t* count);
-/* [host-only] UPGMA G0 (5.1.3 L1287-1295, S19) from codes[n][L] in {0..3}. */
+/* [host-only] UPGMA G0 (5.1.3 L1287-1295, S19) from codes[n][L] in {0..3}, or 16 + base-set
+ * mask for an ambiguity code (S24: a site differs when the two sets are disjoint). */
 mpcgs_status mpcgs_upgma(int32_t n_seq, int32_t n_sites, const uint8_t* codes, double theta0,
                          int32_t* parent, double* age);
 /* [host-only] Post-order register schedule of a tree as used by the pruning kernel
@@ -236,7 +243,9 @@ mpcgs_status mpcgs_upgma(int32_t n_seq, int32_t n_sites, const uint8_t* codes, d
  * factors exp(-u t); returns the register need (max stack depth) or < 0 on error. */
 int32_t mpcgs_tree_schedule(int32_t n_seq, const int32_t* parent, const double* age, double mu,
                             uint32_t* op, double* e);
-/* [host-only] Sequential PHYLIP reader: dims, then rows (n*L chars, row-major). */
+/* [host-only] Sequential PHYLIP reader: dims, then rows (n*L chars, row-major).  Accepts ACGT
+ * and the IUPAC ambiguity characters (mpcgs_init rejects the latter unless cfg->ambiguity);
+ * anything else -> MPCGS_E_ALIGNMENT. */
 mpcgs_status mpcgs_phylip_dims(const char* path, int32_t* n_seq, int32_t* n_sites);
 mpcgs_status mpcgs_phylip_read(const char* path, char* seqs, int32_t cap_chars);
 /* [host-only] Philox4x32-10 block (for known-answer checks of the device generator). */

@@ -151,7 +151,8 @@ struct DevState {
                            // (F84, HKY85: SURVEY 8(f) f4), branch data (t, 0), P(t) from gm
     const double* gm;      // [36] ev[4], V[16], W[16]: P(t) = V diag(exp(ev t)) W (model 1)
     void* sched_P;         // [Nmax][nops][32] P of each op's two children (model 1)
-    const uint8_t* codes;  // [n][Lpad], 0..3
+    int amb;               // 1: codes are base-set masks 1..15 (ambiguity codes, f4 / S24)
+    const uint8_t* codes;  // [n][Lpad], 0..3 (or masks when amb)
     const double* site_w;  // [L] pattern counts when sites are compressed patterns (f3), else nullptr
     // generator (chain state)
     int32_t *parent, *left, *right, *need;  // [nn] (left/right/need valid for interior)

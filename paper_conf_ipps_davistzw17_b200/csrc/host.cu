@@ -362,15 +362,35 @@ double host_S(int n, const double* age) {
     return S;
 }
 
-int code_of(char ch) {
+// A, C, G, T -> 0..3 (S2).  With ambiguity codes (f4, S24): IUPAC letters, '-'
+// and '?' -> 16 + base-set mask (bit X = base X), else -1.
+int code_of(char ch, bool ambiguity = false) {
     switch (ch) {
         case 'A': case 'a': return 0;
         case 'C': case 'c': return 1;
         case 'G': case 'g': return 2;
         case 'T': case 't': return 3;
+        default: break;
+    }
+    if (!ambiguity) return -1;
+    switch (ch) {
+        case 'M': case 'm': return 16 + 3;   // A C
+        case 'R': case 'r': return 16 + 5;   // A G
+        case 'W': case 'w': return 16 + 9;   // A T
+        case 'S': case 's': return 16 + 6;   // C G
+        case 'Y': case 'y': return 16 + 10;  // C T
+        case 'K': case 'k': return 16 + 12;  // G T
+        case 'V': case 'v': return 16 + 7;   // A C G
+        case 'H': case 'h': return 16 + 11;  // A C T
+        case 'D': case 'd': return 16 + 13;  // A G T
+        case 'B': case 'b': return 16 + 14;  // C G T
+        case 'N': case 'n': case '-': case '?': return 16 + 15;
         default: return -1;
     }
 }
+
+// base set of a code: one bit for A..T, the mask for an ambiguity code
+inline int base_set(int code) { return code < 4 ? 1 << code : code - 16; }
 
 // UPGMA (5.1.3 L1287-1295): Hamming distances, average linkage over leaf pairs,
 // node height theta0 * d / 2 forced 1e-6 theta0 above the children (S19).
@@ -382,7 +402,7 @@ void upgma(int n, int L, const uint8_t* codes, double theta0, int32_t* parent, d
             long diff = 0;
             const uint8_t* a = codes + (size_t)i * L;
             const uint8_t* b = codes + (size_t)j * L;
-            for (int s = 0; s < L; ++s) diff += a[s] != b[s];
+            for (int s = 0; s < L; ++s) diff += (base_set(a[s]) & base_set(b[s])) == 0;  // disjoint sets (S24)
             d[i][j] = d[j][i] = (double)diff;
         }
     std::vector<int> live(n), size(nn, 1);
@@ -442,6 +462,7 @@ PruneArgs prune_args(mpcgs_ctx* c, int ntrees_global, double* out, int out_first
     a.sched_op = c->s.sched_op;
     a.sched_e = c->s.sched_e;
     a.gm = c->model ? c->s.gm : nullptr;
+    a.amb = c->s.amb;
     a.sched_P = c->s.sched_P;
     prune_tiling(c->n, c->L, ntrees_global, c->precision, a.tiles, a.sites_per_cta);
     a.tree_need = c->s.tree_need;
@@ -723,7 +744,7 @@ mpcgs_status mpcgs_phylip_read(const char* path, char* seqs, int32_t cap) {
             for (char ch : s) {
                 if (ch == ' ' || ch == '\t' || ch == '\r') continue;
                 if (got >= L) return false;
-                if (code_of(ch) < 0) return false;
+                if (code_of(ch, true) < 0) return false;  // mpcgs_init decides on ambiguity codes
                 seqs[(size_t)r * L + got++] = ch;
             }
             return true;
@@ -760,14 +781,16 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
     if (cfg->precision != 32 && cfg->precision != 64) return MPCGS_E_ARG;
     if (cfg->max_proposals < 1 || cfg->max_proposals > MPCGS_MAX_PROPOSALS || cfg->max_samples < 0) return MPCGS_E_ARG;
     if (cfg->world < 1 || cfg->rank < 0 || cfg->rank >= cfg->world || cfg->burnin_steps < 0) return MPCGS_E_ARG;
-    // alignment -> codes (S2: ACGT only)
+    // alignment -> codes (S2: ACGT only; with cfg->ambiguity also IUPAC sets, S24)
     std::vector<uint8_t> codes((size_t)n * L);
+    bool any_amb = false;
     for (int i = 0; i < n; ++i) {
         if (!aln->rows[i]) return MPCGS_E_ARG;
         for (int s = 0; s < L; ++s) {
-            int cd = code_of(aln->rows[i][s]);
+            int cd = code_of(aln->rows[i][s], cfg->ambiguity != 0);
             if (cd < 0) return MPCGS_E_ALIGNMENT;
             codes[(size_t)i * L + s] = (uint8_t)cd;
+            any_amb |= cd >= 16;
         }
     }
     mpcgs_ctx* c = new mpcgs_ctx();
@@ -790,9 +813,10 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
     bool emp = false;
     for (int i = 0; i < 4; ++i) emp |= cfg->base_freq[i] < 0.0;
     if (emp) {
-        double cnt[4] = {0, 0, 0, 0};
-        for (uint8_t x : codes) cnt[x] += 1.0;
-        for (int i = 0; i < 4; ++i) pi[i] = cnt[i] / ((double)n * L);
+        double cnt[4] = {0, 0, 0, 0}, known = 0.0;
+        for (uint8_t x : codes)
+            if (x < 4) { cnt[x] += 1.0; known += 1.0; }  // ambiguity codes not counted (S24)
+        for (int i = 0; i < 4; ++i) pi[i] = known > 0.0 ? cnt[i] / known : 0.25;
     } else {
         double sum = 0.0;
         for (int i = 0; i < 4; ++i) { pi[i] = cfg->base_freq[i]; sum += pi[i]; }
@@ -944,19 +968,27 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
         s.Mmax = c->Mmax;
         c->theta_cnt = (unsigned*)(b + y.theta_cnt);
         c->score_out = (double*)(b + y.score_out);
-        c->codes2 = (uint32_t*)(b + y.codes2);
+        c->codes2 = any_amb ? nullptr : (uint32_t*)(b + y.codes2);  // 2-bit codes: unambiguous data only
+        s.amb = any_amb ? 1 : 0;
         s.site_w = cfg->compress_patterns ? (const double*)(b + y.site_w) : nullptr;
         if ((st = enter(c))) break;
         if (cudaMemsetAsync(c->ws, 0, y.total, c->work) != cudaSuccess) { st = fail(c, MPCGS_E_CUDA, "memset"); break; }
         std::vector<uint8_t> padded((size_t)n * c->Lpad, 0);
-        for (int i = 0; i < n; ++i) std::memcpy(padded.data() + (size_t)i * c->Lpad, codes.data() + (size_t)i * L, L);
+        // byte codes: bases 0..3, or base-set masks 1..15 when the data hold ambiguity codes
+        for (int i = 0; i < n; ++i)
+            for (int site = 0; site < L; ++site) {
+                const int cd = codes[(size_t)i * L + site];
+                padded[(size_t)i * c->Lpad + site] = (uint8_t)(any_amb ? base_set(cd) : cd);
+            }
         const int W2 = codes2_words(L);
         std::vector<uint32_t> packed((size_t)n * W2, 0u);
-        for (int i = 0; i < n; ++i)
-            for (int site = 0; site < L; ++site)
-                packed[(size_t)i * W2 + (site >> 4)] |= (uint32_t)codes[(size_t)i * L + site] << (2 * (site & 15));
+        if (!any_amb)
+            for (int i = 0; i < n; ++i)
+                for (int site = 0; site < L; ++site)
+                    packed[(size_t)i * W2 + (site >> 4)] |= (uint32_t)codes[(size_t)i * L + site] << (2 * (site & 15));
         if (cudaMemcpyAsync((void*)s.codes, padded.data(), padded.size(), cudaMemcpyHostToDevice, c->work) != cudaSuccess ||
-            cudaMemcpyAsync(c->codes2, packed.data(), packed.size() * 4, cudaMemcpyHostToDevice, c->work) != cudaSuccess) {
+            (c->codes2 &&
+             cudaMemcpyAsync(c->codes2, packed.data(), packed.size() * 4, cudaMemcpyHostToDevice, c->work) != cudaSuccess)) {
             st = fail(c, MPCGS_E_CUDA, "codes upload");
             break;
         }

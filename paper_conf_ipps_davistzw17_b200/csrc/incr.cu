@@ -28,10 +28,11 @@ template <typename T>
 __device__ __forceinline__ int load_node(const DevState& s, int c, int site, T (&v)[4]) {
     if (c < s.n) {
         const int x = __ldg(s.codes + (size_t)c * s.Lpad + site);
-        v[0] = x == 0 ? T(1) : T(0);
-        v[1] = x == 1 ? T(1) : T(0);
-        v[2] = x == 2 ? T(1) : T(0);
-        v[3] = x == 3 ? T(1) : T(0);
+        const int m = s.amb ? x : 1 << x;  // base-set indicator (ambiguity codes: S24)
+        v[0] = (m & 1) ? T(1) : T(0);
+        v[1] = (m & 2) ? T(1) : T(0);
+        v[2] = (m & 4) ? T(1) : T(0);
+        v[3] = (m & 8) ? T(1) : T(0);
         return 0;
     }
     const size_t i = (size_t)(c - s.n) * s.Lg + site;

@@ -30,6 +30,7 @@ struct PruneArgs {
     const void* sched_e;       // [ntrees][nops] float4 / double4
     const double* gm;          // general model (f4): [36] eigen-system of Q, else nullptr (F81)
     void* sched_P;             // general model: [ntrees][nops][32] P matrices (float / double)
+    int amb;                   // byte codes are base-set masks (ambiguity codes): flat kernel only
     int tiles, sites_per_cta;
     const double* site_w;      // [L] pattern counts (compressed sites, f3) or nullptr
     const int32_t* tree_need;  // [ntrees] register need of each tree's schedule (nullable)

@@ -23,7 +23,22 @@
 
 namespace mpcgs {
 
-template <typename T, int D, int S>
+// tip vector of an F81 tip child: base x (0..3), or base-set mask x (AMB, S24):
+// v_X = e [X in set] + em pi(set)
+template <typename T, bool AMB>
+__device__ __forceinline__ void tip81(T (&r)[4], int x, T e, T em, const T (&pi)[4]) {
+    if constexpr (AMB) {
+        const T ps = ((x & 1) ? pi[0] : T(0)) + ((x & 2) ? pi[1] : T(0)) + ((x & 4) ? pi[2] : T(0)) +
+                     ((x & 8) ? pi[3] : T(0));
+        const T c = em * ps;
+#pragma unroll
+        for (int i = 0; i < 4; ++i) r[i] = ((x >> i) & 1) ? c + e : c;
+    } else {
+        tipvec<T>(r, x, e, em, pi);
+    }
+}
+
+template <typename T, int D, int S, bool AMB>
 __device__ __forceinline__ void op_tt(T (&R)[D][4], uint32_t code, const typename Traits<T>::E4& ed,
                                       const uint8_t* __restrict__ codes, int Lpad, int site,
                                       const T (&pi)[4], int& scale) {
@@ -32,15 +47,15 @@ __device__ __forceinline__ void op_tt(T (&R)[D][4], uint32_t code, const typenam
         int xa = __ldg(codes + (size_t)ta * Lpad + site);
         int xb = __ldg(codes + (size_t)tb * Lpad + site);
         T va[4], vb[4];
-        tipvec<T>(va, xa, ed.x, ed.y, pi);
-        tipvec<T>(vb, xb, ed.z, ed.w, pi);
+        tip81<T, AMB>(va, xa, ed.x, ed.y, pi);
+        tip81<T, AMB>(vb, xb, ed.z, ed.w, pi);
 #pragma unroll
         for (int i = 0; i < 4; ++i) R[S][i] = va[i] * vb[i];
         maybe_rescale(R[S], scale);
     }
 }
 
-template <typename T, int D, int S>
+template <typename T, int D, int S, bool AMB>
 __device__ __forceinline__ void op_ts(T (&R)[D][4], uint32_t code, const typename Traits<T>::E4& ed,
                                       const uint8_t* __restrict__ codes, int Lpad, int site,
                                       const T (&pi)[4], int& scale) {
@@ -48,7 +63,7 @@ __device__ __forceinline__ void op_ts(T (&R)[D][4], uint32_t code, const typenam
         int ta = (code >> 6) & 2047;
         int xa = __ldg(codes + (size_t)ta * Lpad + site);
         T va[4];
-        tipvec<T>(va, xa, ed.x, ed.y, pi);
+        tip81<T, AMB>(va, xa, ed.x, ed.y, pi);
         branch<T>(R[S - 1], ed.z, ed.w, pi);
 #pragma unroll
         for (int i = 0; i < 4; ++i) R[S - 1][i] *= va[i];
@@ -71,10 +86,17 @@ __device__ __forceinline__ void op_ss(T (&R)[D][4], const typename Traits<T>::E4
 // ---- general reversible model: per-op P matrices {P_a, P_b}
 // (row-major, row = parent state) formed by k_pmat; the tip vector of state x is
 // column x of P (Eq. 19 with a one-hot child partial), a branch is P . R.
-template <typename T>
+template <typename T, bool AMB>
 __device__ __forceinline__ void gm_tip(T (&v)[4], const T* __restrict__ P, int x) {
+    if constexpr (AMB) {  // base-set mask: sum of the set's columns (S24)
 #pragma unroll
-    for (int i = 0; i < 4; ++i) v[i] = __ldg(P + i * 4 + x);
+        for (int i = 0; i < 4; ++i)
+            v[i] = ((x & 1) ? __ldg(P + i * 4) : T(0)) + ((x & 2) ? __ldg(P + i * 4 + 1) : T(0)) +
+                   ((x & 4) ? __ldg(P + i * 4 + 2) : T(0)) + ((x & 8) ? __ldg(P + i * 4 + 3) : T(0));
+    } else {
+#pragma unroll
+        for (int i = 0; i < 4; ++i) v[i] = __ldg(P + i * 4 + x);
+    }
 }
 
 template <typename T>
@@ -91,27 +113,27 @@ __device__ __forceinline__ void gm_branch(T (&R)[4], const T* __restrict__ P) {
     for (int i = 0; i < 4; ++i) R[i] = o[i];
 }
 
-template <typename T, int D, int S>
+template <typename T, int D, int S, bool AMB>
 __device__ __forceinline__ void gm_tt(T (&R)[D][4], uint32_t code, const T* __restrict__ P,
                                       const uint8_t* __restrict__ codes, int Lpad, int site, int& scale) {
     if constexpr (S < D) {
         int ta = (code >> 6) & 2047, tb = (code >> 17) & 2047;
         T va[4], vb[4];
-        gm_tip<T>(va, P, __ldg(codes + (size_t)ta * Lpad + site));
-        gm_tip<T>(vb, P + 16, __ldg(codes + (size_t)tb * Lpad + site));
+        gm_tip<T, AMB>(va, P, __ldg(codes + (size_t)ta * Lpad + site));
+        gm_tip<T, AMB>(vb, P + 16, __ldg(codes + (size_t)tb * Lpad + site));
 #pragma unroll
         for (int i = 0; i < 4; ++i) R[S][i] = va[i] * vb[i];
         maybe_rescale(R[S], scale);
     }
 }
 
-template <typename T, int D, int S>
+template <typename T, int D, int S, bool AMB>
 __device__ __forceinline__ void gm_ts(T (&R)[D][4], uint32_t code, const T* __restrict__ P,
                                       const uint8_t* __restrict__ codes, int Lpad, int site, int& scale) {
     if constexpr (S >= 1 && S <= D) {
         int ta = (code >> 6) & 2047;
         T va[4];
-        gm_tip<T>(va, P, __ldg(codes + (size_t)ta * Lpad + site));
+        gm_tip<T, AMB>(va, P, __ldg(codes + (size_t)ta * Lpad + site));
         gm_branch<T>(R[S - 1], P + 16);
 #pragma unroll
         for (int i = 0; i < 4; ++i) R[S - 1][i] *= va[i];
@@ -131,8 +153,8 @@ __device__ __forceinline__ void gm_ss(T (&R)[D][4], const T* __restrict__ P, int
 }
 
 #define MPCGS_GMCASE(S)                                                                       \
-    case (OP_TT | ((S) << 2)): gm_tt<T, D, S>(R, code, P, codes, Lpad, site, scale); break; \
-    case (OP_TS | ((S) << 2)): gm_ts<T, D, S>(R, code, P, codes, Lpad, site, scale); break; \
+    case (OP_TT | ((S) << 2)): gm_tt<T, D, S, AMB>(R, code, P, codes, Lpad, site, scale); break; \
+    case (OP_TS | ((S) << 2)): gm_ts<T, D, S, AMB>(R, code, P, codes, Lpad, site, scale); break; \
     case (OP_SS | ((S) << 2)): gm_ss<T, D, S>(R, P, scale); break;
 
 // P matrices of every op's two children from the branch lengths in sched_e
@@ -155,11 +177,11 @@ __global__ void __launch_bounds__(128) k_pmat(const void* sched_e, const double*
 }
 
 #define MPCGS_OPCASE(S)                                                                     \
-    case (OP_TT | ((S) << 2)): op_tt<T, D, S>(R, code, ed, codes, Lpad, site, pi, scale); break; \
-    case (OP_TS | ((S) << 2)): op_ts<T, D, S>(R, code, ed, codes, Lpad, site, pi, scale); break; \
+    case (OP_TT | ((S) << 2)): op_tt<T, D, S, AMB>(R, code, ed, codes, Lpad, site, pi, scale); break; \
+    case (OP_TS | ((S) << 2)): op_ts<T, D, S, AMB>(R, code, ed, codes, Lpad, site, pi, scale); break; \
     case (OP_SS | ((S) << 2)): op_ss<T, D, S>(R, ed, pi, scale); break;
 
-template <typename T, int D, bool W, bool GM>
+template <typename T, int D, bool W, bool GM, bool AMB>
 __global__ void __launch_bounds__(PRUNE_THREADS) k_prune(PruneArgs a) {
     using E4 = typename Traits<T>::E4;
     extern __shared__ __align__(16) unsigned char smem_raw[];
@@ -675,10 +697,10 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
     }
 }
 
-template <typename T, int D, bool W, bool GM>
+template <typename T, int D, bool W, bool GM, bool AMB>
 static cudaError_t launch_flat_w(const PruneArgs& a, int ntrees, cudaStream_t st) {
     size_t smem = (size_t)a.nops * (sizeof(typename Traits<T>::E4) + sizeof(uint32_t));
-    auto kern = k_prune<T, D, W, GM>;
+    auto kern = k_prune<T, D, W, GM, AMB>;
     static size_t attr_bytes = 48 * 1024;  // raised once, outside graph capture (first launch is at init)
     if (smem > attr_bytes) {
         cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
@@ -692,7 +714,11 @@ static cudaError_t launch_flat_w(const PruneArgs& a, int ntrees, cudaStream_t st
 
 template <typename T, int D, bool GM>
 static cudaError_t launch_flat(const PruneArgs& a, int ntrees, cudaStream_t st) {
-    return a.site_w ? launch_flat_w<T, D, true, GM>(a, ntrees, st) : launch_flat_w<T, D, false, GM>(a, ntrees, st);
+    if (a.amb)
+        return a.site_w ? launch_flat_w<T, D, true, GM, true>(a, ntrees, st)
+                        : launch_flat_w<T, D, false, GM, true>(a, ntrees, st);
+    return a.site_w ? launch_flat_w<T, D, true, GM, false>(a, ntrees, st)
+                    : launch_flat_w<T, D, false, GM, false>(a, ntrees, st);
 }
 
 template <typename T, int DR, int SI, bool PT, int DMX, bool W, bool GM>

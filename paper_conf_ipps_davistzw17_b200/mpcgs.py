@@ -40,6 +40,7 @@ class mpcgs_config(ctypes.Structure):
         ("nccl_id", ctypes.c_void_p), ("stream", ctypes.c_void_p), ("workspace", ctypes.c_void_p),
         ("workspace_bytes", ctypes.c_size_t), ("incremental", ctypes.c_int32),
         ("compress_patterns", ctypes.c_int32), ("model", ctypes.c_int32), ("kappa", ctypes.c_double),
+        ("ambiguity", ctypes.c_int32),
     ]
 
 
@@ -215,7 +216,7 @@ class Context:
     def __init__(self, rows, theta0, *, precision=64, burnin_steps=0, max_proposals=1024,
                  max_samples=1 << 20, base_freq=None, mu=0.0, init_tree=None, rank=0, world=1,
                  nccl_id=None, stream=None, workspace=None, phylip=None, incremental=False,
-                 compress_patterns=False, model="F81", kappa=0.0):
+                 compress_patterns=False, model="F81", kappa=0.0, ambiguity=False):
         L = lib()
         cfg = mpcgs_config()
         L.mpcgs_config_default(ctypes.byref(cfg))
@@ -231,6 +232,7 @@ class Context:
         cfg.compress_patterns = int(bool(compress_patterns))
         cfg.model = MODELS[model] if isinstance(model, str) else int(model)
         cfg.kappa = float(kappa)
+        cfg.ambiguity = int(bool(ambiguity))
         self._keep = []
         if init_tree is not None:
             p = _i32a(init_tree[0])

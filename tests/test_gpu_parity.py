@@ -84,6 +84,47 @@ def test_lockstep_general_model_compressed_fp32(P, orc):
     _lockstep(P, orc, wl, 16, 10, wl["chain_seed"], precision=32, compress=True, model="HKY85", kappa=3.0)
 
 
+@pytest.mark.parametrize("model,kappa", [("F81", 0.0), ("HKY85", 4.0)])
+@pytest.mark.parametrize("precision", [64, 32])
+@pytest.mark.parametrize("n,L", [(3, 7), (12, 1000), (64, 300), (256, 500)])
+def test_score_trees_ambiguity_codes(P, orc, model, kappa, precision, n, L):
+    """SURVEY 8(f) f4 / reading S24: IUPAC ambiguity codes and gaps as base-set
+    indicator tips (flat kernel with mask codes) against the oracle."""
+    rng = np.random.default_rng(13 * n + L)
+    pi = np.array([0.22, 0.28, 0.31, 0.19])
+    true_p, true_a = synth.coalescent_tree(n, 0.05, rng)
+    codes = synth.ambiguate(synth.f81_alignment(true_p, true_a, L, pi, orc.default_rate(pi), rng), 0.15, rng,
+                            gap_frac=0.1)
+    trees = [synth.coalescent_tree(n, th, rng) for th in (0.01, 0.3)]
+    trees += [synth.shaped_tree(n, s, rng, scale=0.02) for s in ("caterpillar", "balanced")]
+    u = orc.default_rate(pi)
+    ctx = _ctx(P, codes, 0.05, tree=trees[0], precision=precision, base_freq=pi, mu=u, max_proposals=8,
+               max_samples=16, model=model, kappa=kappa, ambiguity=True)
+    got = ctx.mpcgs_score_trees(np.stack([t[0] for t in trees]), np.stack([t[1] for t in trees]))
+    for (p, a), g in zip(trees, got):
+        if model == "F81":
+            want = orc.log_likelihood(codes, p, a, pi, u)
+        else:
+            want = orc.log_likelihood_model(model, kappa, codes, p, a, pi)
+        assert abs(g - want) <= LL_TOL[precision] * abs(want), (g, want)
+
+
+@pytest.mark.parametrize("incremental,compress,model", [(False, False, "F81"), (True, False, "F81"),
+                                                        (False, True, "F81"), (False, False, "F84")])
+def test_lockstep_ambiguity_codes(P, orc, incremental, compress, model):
+    wl = dict(synth.workload("c2", L=300))
+    wl["codes"] = synth.ambiguate(wl["codes"], 0.1, np.random.default_rng(4), gap_frac=0.05)
+    assert _lockstep(P, orc, wl, 32, 8, wl["chain_seed"], incremental=incremental, compress=compress,
+                     model=model, kappa=2.0 if model != "F81" else 0.0, ambiguity=True) <= 2
+
+
+def test_ambiguity_off_rejects_iupac(P):
+    with pytest.raises(P.MpcgsError):
+        P.Context(["ACGT", "ACGN", "ACGA"], 0.1, max_proposals=4, max_samples=4)
+    ctx = P.Context(["ACGT", "ACGN", "AC-A"], 0.1, max_proposals=4, max_samples=4, ambiguity=True)
+    ctx.free()
+
+
 def test_general_model_argument_errors(P):
     rows = ["ACGT", "ACGA", "ACGG"]
     with pytest.raises(P.MpcgsError):
@@ -138,7 +179,7 @@ def test_underflow_rescaling_long_alignment_many_tips(P, orc):
 
 # ------------------------------------------------------------------ GMH step (lock-step, P20)
 def _lockstep(P, orc, wl, N, steps, seed, K=None, precision=64, incremental=False, compress=False,
-              model="F81", kappa=0.0):
+              model="F81", kappa=0.0, ambiguity=False):
     codes = wl["codes"]
     pi = orc.base_freqs(codes)
     u = orc.default_rate(pi)
@@ -149,7 +190,8 @@ def _lockstep(P, orc, wl, N, steps, seed, K=None, precision=64, incremental=Fals
     else:
         gl = orc.log_likelihood_model(model, kappa, codes, parent, age, pi)
     ctx = _ctx(P, codes, theta0, tree=(parent, age), precision=precision, max_proposals=N, max_samples=16,
-               incremental=incremental, compress_patterns=compress, model=model, kappa=kappa)
+               incremental=incremental, compress_patterns=compress, model=model, kappa=kappa,
+               ambiguity=ambiguity)
     K = N if K is None else K
     height = age.max()
     skipped = 0

@@ -66,10 +66,23 @@ def test_phylip_reader(tmp_path):
     f.write_text("3 8\nalpha     ACGTACGT\nb ACGT ACGT\nc_long_nam\nacgtacgt\n")
     rows = P.mpcgs_phylip_read(str(f))
     assert rows == ["ACGTACGT", "ACGTACGT", "acgtacgt"]
+    amb = tmp_path / "amb.phy"  # IUPAC characters are read; mpcgs_init decides (S2 / S24)
+    amb.write_text("2 4\na ACGN\nb AC-R\n")
+    assert P.mpcgs_phylip_read(str(amb)) == ["ACGN", "AC-R"]
     bad = tmp_path / "bad.phy"
-    bad.write_text("2 4\na ACGN\nb ACGT\n")
+    bad.write_text("2 4\na ACGX\nb ACGT\n")
     with pytest.raises(P.MpcgsError):
         P.mpcgs_phylip_read(str(bad))
+
+
+def test_upgma_ambiguity_sets_match_oracle(orc):
+    rng = np.random.default_rng(3)
+    wl = synth.workload("c2")
+    codes = synth.ambiguate(wl["codes"], 0.2, rng, gap_frac=0.05)
+    p1, a1 = P.mpcgs_upgma(codes, wl["theta0"])
+    p2, a2 = orc.upgma(codes, wl["theta0"])
+    assert np.array_equal(p1, p2)
+    assert np.allclose(a1, a2, rtol=1e-15)
 
 
 def _interpret(op, e, codes, pi):
