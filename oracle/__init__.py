@@ -97,6 +97,11 @@ def lib():
         L.orc_theta_hat.argtypes = [c.c_int, _f64p, c.c_int, c.c_double, c.c_int, c.c_void_p,
                                     c.c_void_p]
         L.orc_theta_hat.restype = c.c_double
+        L.orc_log_rel_likelihood_loci.argtypes = [c.c_int, _i32p, _f64p, _i32p, _f64p, c.c_double]
+        L.orc_log_rel_likelihood_loci.restype = c.c_double
+        L.orc_theta_hat_loci.argtypes = [c.c_int, _i32p, _f64p, _i32p, _f64p, c.c_int, c.c_void_p,
+                                         c.c_void_p]
+        L.orc_theta_hat_loci.restype = c.c_double
         L.orc_theta_alg2.argtypes = [c.c_int, _f64p, c.c_int, c.c_double, c.c_int]
         L.orc_theta_alg2.restype = c.c_double
         L.orc_upgma.argtypes = [c.c_int, c.c_int, _u8p, c.c_double, _i32p, _f64p]
@@ -316,6 +321,24 @@ def theta_hat(S, n, theta0, G=4096, curve=False):
     S = np.ascontiguousarray(S, np.float64)
     gt, gl = np.zeros(G), np.zeros(G)
     th = lib().orc_theta_hat(len(S), S, n, theta0, G, gt.ctypes.data, gl.ctypes.data)
+    return (th, gt, gl) if curve else th
+
+
+def _loci(S_list, n_list, theta0_list):
+    M = np.array([len(x) for x in S_list], np.int32)
+    S = np.ascontiguousarray(np.concatenate([np.asarray(x, np.float64) for x in S_list]))
+    return (len(S_list), M, S, np.ascontiguousarray(n_list, np.int32),
+            np.ascontiguousarray(theta0_list, np.float64))
+
+
+def log_rel_likelihood_loci(S_list, n_list, theta0_list, theta):
+    """Joint ln L(theta) of independent loci sharing theta."""
+    return lib().orc_log_rel_likelihood_loci(*_loci(S_list, n_list, theta0_list), theta)
+
+
+def theta_hat_loci(S_list, n_list, theta0_list, G=4096, curve=False):
+    gt, gl = np.zeros(G), np.zeros(G)
+    th = lib().orc_theta_hat_loci(*_loci(S_list, n_list, theta0_list), G, gt.ctypes.data, gl.ctypes.data)
     return (th, gt, gl) if curve else th
 
 

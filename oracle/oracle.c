@@ -1024,6 +1024,94 @@ double orc_theta_hat(int M, const double* S, int n, double theta0, int G,
 }
 
 /*
+ * Multiple loci: loci with independent genealogies share theta, so
+ * the joint relative likelihood is the product over loci of Eq. 25 (L765-797), each
+ * locus l with its own samples S_l[0..M_l), n_l and driving value theta0_l.  The
+ * samples are concatenated: locus l starts at sum_{k<l} M_k.
+ */
+double orc_log_rel_likelihood_loci(int K, const int* M, const double* S, const int* n,
+                                   const double* theta0, double theta) {
+    double r = 0.0;
+    int l;
+    long off = 0;
+    for (l = 0; l < K; ++l) {
+        r += orc_log_rel_likelihood(M[l], S + off, n[l], theta0[l], theta);
+        off += M[l];
+    }
+    return r;
+}
+
+/* d ln L / d theta = sum_l (S_w,l(theta) - (n_l - 1) theta) / theta^2: the sign of the sum */
+static double stationarity_loci(int K, const int* M, const double* S, const int* n,
+                                const double* theta0, double theta) {
+    double f = 0.0;
+    int l;
+    long off = 0;
+    for (l = 0; l < K; ++l) {
+        f += stationarity(M[l], S + off, n[l], theta0[l], theta);
+        off += M[l];
+    }
+    return f;
+}
+
+/* Joint theta-hat: global argmax over [sum_l S_min,l, sum_l S_max,l] / sum_l (n_l - 1)
+   (every stationary point solves sum_l S_w,l = theta sum_l (n_l - 1)), by the same
+   grid + bisection (else golden section) as orc_theta_hat. */
+double orc_theta_hat_loci(int K, const int* M, const double* S, const int* n,
+                          const double* theta0, int G, double* grid_theta, double* grid_ll) {
+    double smin = 0.0, smax = 0.0, dof = 0.0, lo, hi, best_ll = -INFINITY, a0, a1;
+    int g, l, best = 0, it;
+    long off = 0;
+    for (l = 0; l < K; ++l) {
+        double mn = INFINITY, mx = -INFINITY;
+        for (g = 0; g < M[l]; ++g) {
+            if (S[off + g] < mn) mn = S[off + g];
+            if (S[off + g] > mx) mx = S[off + g];
+        }
+        smin += mn;
+        smax += mx;
+        dof += (double)(n[l] - 1);
+        off += M[l];
+    }
+    a0 = smin / dof;
+    a1 = smax / dof;
+    if (a0 == a1 || G < 3) return a0;
+    for (g = 0; g < G; ++g) {
+        double th = exp(log(a0) + (log(a1) - log(a0)) * g / (G - 1));
+        double ll = orc_log_rel_likelihood_loci(K, M, S, n, theta0, th);
+        if (grid_theta) grid_theta[g] = th;
+        if (grid_ll) grid_ll[g] = ll;
+        if (ll > best_ll) {
+            best_ll = ll;
+            best = g;
+        }
+    }
+    lo = best > 0 ? exp(log(a0) + (log(a1) - log(a0)) * (best - 1) / (G - 1)) : a0;
+    hi = best < G - 1 ? exp(log(a0) + (log(a1) - log(a0)) * (best + 1) / (G - 1)) : a1;
+    if (stationarity_loci(K, M, S, n, theta0, lo) >= 0.0 &&
+        stationarity_loci(K, M, S, n, theta0, hi) <= 0.0) {
+        for (it = 0; it < 200 && hi - lo > 1e-15 * hi; ++it) {
+            double mid = 0.5 * (lo + hi);
+            if (stationarity_loci(K, M, S, n, theta0, mid) >= 0.0) lo = mid;
+            else hi = mid;
+        }
+        return 0.5 * (lo + hi);
+    }
+    {
+        const double gr = 0.6180339887498949;
+        double a = lo, b = hi, c = b - gr * (b - a), d = a + gr * (b - a);
+        for (it = 0; it < 300 && b - a > 1e-15 * b; ++it) {
+            if (orc_log_rel_likelihood_loci(K, M, S, n, theta0, c) >
+                orc_log_rel_likelihood_loci(K, M, S, n, theta0, d)) b = d;
+            else a = c;
+            c = b - gr * (b - a);
+            d = a + gr * (b - a);
+        }
+        return 0.5 * (a + b);
+    }
+}
+
+/*
  * Algorithm 2 (L1329-1340) literally, on ln L, with delta = 1e-6 theta0 and
  * eps = 1e-9 theta0 (S20).  A cross-check only: a local ascent from theta0.
  */

@@ -108,6 +108,12 @@ double orc_weighted_mean_S(int M, const double* S, double theta0, double theta);
 double orc_em_map(int M, const double* S, int n, double theta0, double theta);
 double orc_theta_hat(int M, const double* S, int n, double theta0, int G,
                      double* grid_theta, double* grid_ll);
+/* Multiple loci sharing theta: product of Eq. 25 over loci; samples
+   of locus l at S[sum_{k<l} M_k ...] */
+double orc_log_rel_likelihood_loci(int K, const int* M, const double* S, const int* n,
+                                   const double* theta0, double theta);
+double orc_theta_hat_loci(int K, const int* M, const double* S, const int* n,
+                          const double* theta0, int G, double* grid_theta, double* grid_ll);
 double orc_theta_alg2(int M, const double* S, int n, double theta0, int max_iter);
 
 /* Initial genealogy G0 by UPGMA (5.1.3 L1287-1295; reading S19) */

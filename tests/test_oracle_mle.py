@@ -89,3 +89,45 @@ def test_synthetic_workload_shapes():
         wl = synth.workload(name)
         assert wl["codes"].shape == (n, L)
         assert wl["codes"].dtype == np.uint8 and wl["codes"].max() <= 3
+
+
+# ------------------------------------------------------------------ multiple loci
+def test_loci_one_locus_is_single_locus(orc):
+    rng = np.random.default_rng(2)
+    S = rng.gamma(3.0, 0.02, 500)
+    assert orc.theta_hat_loci([S], [12], [0.01]) == orc.theta_hat(S, 12, 0.01)
+    for th in (0.003, 0.01, 0.05):
+        assert orc.log_rel_likelihood_loci([S], [12], [0.01], th) == orc.log_rel_likelihood(S, 12, 0.01, th)
+
+
+def test_loci_degenerate_closed_form(orc):
+    """One value of S per locus: ln L = sum_l (n_l-1) ln(theta0_l/theta) - S_l (1/theta - 1/theta0_l),
+    maximised at sum_l S_l / sum_l (n_l - 1) (differentiate); the grid + bisection must find it."""
+    S_list = [np.full(7, 0.3), np.full(3, 1.1), np.full(5, 0.05)]
+    n_list, t0 = [5, 12, 4], [0.01, 0.02, 0.005]
+    want = (0.3 + 1.1 + 0.05) / (4 + 11 + 3)
+    assert abs(orc.theta_hat_loci(S_list, n_list, t0) - want) <= 1e-13 * want
+
+
+def test_loci_product_stationarity_and_duplication(orc):
+    rng = np.random.default_rng(9)
+    S_list = [rng.gamma(4.0, 0.01, 300), rng.gamma(2.0, 0.05, 200)]
+    n_list, t0 = [8, 16], [0.01, 0.03]
+    th = orc.theta_hat_loci(S_list, n_list, t0)
+    # the joint likelihood is the product over loci (independent genealogies, one theta)
+    for x in (0.5 * th, th, 2 * th):
+        parts = sum(orc.log_rel_likelihood(S, n, a, x) for S, n, a in zip(S_list, n_list, t0))
+        assert np.isclose(orc.log_rel_likelihood_loci(S_list, n_list, t0, x), parts, rtol=1e-14)
+    # stationarity: sum_l S_w,l(theta-hat) = theta-hat sum_l (n_l - 1)
+    sw = sum(orc.weighted_mean_S(S, a, th) for S, a in zip(S_list, t0))
+    assert abs(sw - th * sum(n - 1 for n in n_list)) <= 1e-9 * sw
+    # bracket, and a duplicated locus set leaves the argmax unchanged
+    lo = sum(S.min() for S in S_list) / sum(n - 1 for n in n_list)
+    hi = sum(S.max() for S in S_list) / sum(n - 1 for n in n_list)
+    assert lo <= th <= hi
+    th2 = orc.theta_hat_loci(S_list * 2, n_list * 2, t0 * 2)
+    assert abs(th2 - th) <= 1e-9 * th
+    # a global maximum on a fine scan
+    xs = np.exp(np.linspace(np.log(lo), np.log(hi), 2001))
+    ll = [orc.log_rel_likelihood_loci(S_list, n_list, t0, x) for x in xs]
+    assert orc.log_rel_likelihood_loci(S_list, n_list, t0, th) >= max(ll) - 1e-12
