@@ -194,6 +194,55 @@ def workload_config(args, wl):
                           "(SURVEY 8(f) f4; flat kernel)" if args.ambiguity > 0 else "none")}
 
 
+def run_loci(args, over):
+    """Auxiliary measurement: K independent loci of the workload's shape
+    (data sweep indices 0..K-1), one context each, sampled concurrently with
+    mpcgs_sample_loci (each locus on its own stream).  Timed with CUDA events on the
+    caller's stream around the whole call (its loops wait on that stream and the call
+    returns after all of them), L2 not flushed; one JSON line, no roofline."""
+    import torch
+
+    import paper_conf_ipps_davistzw17_b200 as P
+
+    K = args.loci
+    wls = [synth.workload(args.workload, sweep=k, theta_true=args.theta_true, **over) for k in range(K)]
+    n, L = wls[0]["codes"].shape
+    N = wls[0]["N"]
+    stream = torch.cuda.current_stream().cuda_stream
+    mk = dict(precision=args.precision, max_proposals=N, stream=stream, model=args.model, kappa=args.kappa,
+              incremental=args.incremental, compress_patterns=args.compress)
+    ctxs = [P.Context(synth.to_strings(w["codes"]), w["theta0"], max_samples=N * max(args.steps, args.warmup),
+                      init_tree=(w["true_parent"], w["true_age"]), **mk) for w in wls]
+    seeds = [w["chain_seed"] for w in wls]
+    P.mpcgs_sample_loci(ctxs, N, N * args.warmup, seeds)
+    torch.cuda.synchronize()
+    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    e0.record()
+    P.mpcgs_sample_loci(ctxs, N, N * args.steps, [x + 1 for x in seeds])
+    e1.record()
+    torch.cuda.synchronize()
+    ms = e0.elapsed_time(e1)
+    one = None
+    if K > 1:  # the same loci one after another, for the overlap factor
+        e0.record()
+        for c, sd in zip(ctxs, seeds):
+            c.mpcgs_sample(N, N * args.steps, sd + 1)
+        e1.record()
+        torch.cuda.synchronize()
+        one = e0.elapsed_time(e1)
+    partials = K * N * L * (n - 1) * args.steps
+    line = {"metric": METRIC, "value": partials / (ms / 1e3), "unit": UNIT, "n_gpus": 1, "steps": args.steps,
+            "warmup": args.warmup, "ms_per_step": ms / args.steps, "higher_is_better": True,
+            "dtype": "f64" if args.precision == 64 else "f32", "data": "synthetic",
+            "config": dict(workload_config(args, wls[0]), loci=K, l2="not flushed (concurrent loci)"),
+            "proposals_per_s": K * N * args.steps / (ms / 1e3),
+            "sequential_ms": one, "overlap_speedup": (one / ms) if one else None, "roofline": None,
+            "note": "auxiliary multi-locus run (SURVEY 8(f) f4): K loci sampled concurrently on one GPU"}
+    print(json.dumps(line), flush=True)
+    for c in ctxs:
+        c.free()
+
+
 def main():
     ap = argparse.ArgumentParser()
     ap.add_argument("--gpus", type=int, default=1)
@@ -220,6 +269,8 @@ def main():
     ap.add_argument("--ambiguity", type=float, default=0.0,
                     help="fraction of characters replaced by IUPAC ambiguity codes (plus half that as N); "
                          "SURVEY 8(f) f4")
+    ap.add_argument("--loci", type=int, default=1,
+                    help="K > 1: auxiliary run of K independent loci sampled concurrently (SURVEY 8(f) f4)")
     args = ap.parse_args()
     args.warmup = max(args.warmup, 3)
 
@@ -241,6 +292,9 @@ def main():
                                       gap_frac=args.ambiguity / 2)
     if args.impl == "reference":
         run_reference(args, wl, rank)
+        return
+    if args.loci > 1:
+        run_loci(args, over)
         return
 
     import torch

@@ -215,6 +215,27 @@ mpcgs_status mpcgs_set_theta0(mpcgs_ctx* ctx, double theta0);
 mpcgs_status mpcgs_em(mpcgs_ctx* ctx, int32_t n_iter, int32_t n_proposals, int64_t n_samples,
                       uint64_t seed, int32_t n_grid, double* theta_trace);
 
+/* Multiple loci: loci have independent genealogies and share theta, so
+ * the joint relative likelihood is the product over loci of Eq. 25 (L765-797).  ctxs: host
+ * array of n_loci contexts (one per locus alignment; any n, L, model; same device).
+ *
+ * mpcgs_sample_loci: mpcgs_sample on every locus with seeds[l] (host [n_loci]); all loops are
+ * enqueued (each on its context's stream) before any is waited for, so loci overlap on the GPU.
+ * Returns the first error; every enqueued loop is finished.
+ * mpcgs_estimate_theta_loci: the global argmax of sum_l ln L_l(theta) over the bracket
+ * [sum_l S_min,l, sum_l S_max,l] / sum_l (n_l - 1) (S20 generalised), grid of n_grid points
+ * (grid_theta / grid_logL: host [n_grid], nullable; grid_logL is the summed curve) then
+ * safeguarded Newton on sum_l (S_w,l(theta) - (n_l - 1) theta).  One locus = mpcgs_estimate_theta.
+ * mpcgs_em_loci: n_iter times { sample_loci(seeds[l] + it); joint theta-hat; every theta0 <- it }.
+ * MPCGS_E_ARG on null / empty arrays; MPCGS_E_STATE if a locus has no samples. */
+mpcgs_status mpcgs_sample_loci(mpcgs_ctx* const* ctxs, int32_t n_loci, int32_t n_proposals,
+                               int64_t n_samples, const uint64_t* seeds);
+mpcgs_status mpcgs_estimate_theta_loci(mpcgs_ctx* const* ctxs, int32_t n_loci, double* theta_hat,
+                                       int32_t n_grid, double* grid_theta, double* grid_logL);
+mpcgs_status mpcgs_em_loci(mpcgs_ctx* const* ctxs, int32_t n_loci, int32_t n_iter,
+                           int32_t n_proposals, int64_t n_samples, const uint64_t* seeds,
+                           int32_t n_grid, double* theta_trace);
+
 /* Model parameters actually used (host out: pi[4], u). */
 mpcgs_status mpcgs_get_model(const mpcgs_ctx* ctx, double* pi, double* mu);
 

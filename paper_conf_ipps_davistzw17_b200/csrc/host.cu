@@ -86,6 +86,15 @@ struct mpcgs_ctx {
     std::vector<cudaEvent_t> evpool;
     cudaEvent_t ev_a = nullptr, ev_b = nullptr;
     std::vector<double> pinned_dummy;
+    // a sampling loop enqueued by sample_begin and not yet finished by sample_end
+    struct {
+        bool active = false;
+        cudaGraph_t graph = nullptr;
+        cudaGraphExec_t exec = nullptr;
+        cudaEvent_t end = nullptr;
+        int N = 0;
+        int64_t M = 0;
+    } pend;
 };
 
 namespace {
@@ -1043,8 +1052,16 @@ mpcgs_status mpcgs_set_timing(mpcgs_ctx* c, int32_t mode) {
     return MPCGS_OK;
 }
 
-mpcgs_status mpcgs_sample(mpcgs_ctx* c, int32_t N, int64_t M, uint64_t seed) {
+}  // extern "C"
+
+namespace {
+// Enqueue burn-in + sampling on the context's stream (timing mode: run and time
+// it); sample_end waits for it.  Loops of several contexts (loci) overlap on the
+// device when they are all begun before any is ended.
+mpcgs_status sample_end(mpcgs_ctx* c);
+mpcgs_status sample_begin(mpcgs_ctx* c, int32_t N, int64_t M, uint64_t seed) {
     CHECK_CTX(c);
+    if (c->pend.active) return fail(c, MPCGS_E_STATE, "a sampling loop is still pending");
     if (N < 1 || N > c->Nmax || N % c->world != 0 || M < 0 || M > c->Mmax)
         return fail(c, MPCGS_E_ARG, "n_proposals / n_samples out of range or not divisible by world");
     if (c->world > 1 && !c->comm)
@@ -1138,23 +1155,70 @@ mpcgs_status mpcgs_sample(mpcgs_ctx* c, int32_t N, int64_t M, uint64_t seed) {
         }
         for (int64_t k = 0; k < rest; ++k)
             if ((st = one_step())) return st;
-        cudaEvent_t ev_end;
-        CU(cudaEventCreate(&ev_end));
-        CU(cudaEventRecord(ev_end, c->work));
-        CU(cudaEventSynchronize(ev_end));
+        c->pend.graph = graph;
+        c->pend.exec = exec;
+        CU(cudaEventCreate(&c->pend.end));
+        CU(cudaEventRecord(c->pend.end, c->work));
+    }
+    c->pend.active = true;
+    c->pend.N = N;
+    c->pend.M = M;
+    return MPCGS_OK;
+}
+
+mpcgs_status sample_end(mpcgs_ctx* c) {
+    CHECK_CTX(c);
+    if (!c->pend.active) return fail(c, MPCGS_E_STATE, "no sampling loop pending");
+    c->pend.active = false;
+    mpcgs_status st = MPCGS_OK;
+    if (c->pend.end) {
+        cudaEvent_t ev_end = c->pend.end;
+        c->pend.end = nullptr;
+        const cudaError_t e1 = cudaEventSynchronize(ev_end);
         float ms = 0.f;
-        CU(cudaEventElapsedTime(&ms, c->ev_b, ev_end));
+        const cudaError_t e2 = e1 == cudaSuccess ? cudaEventElapsedTime(&ms, c->ev_b, ev_end) : e1;
         cudaEventDestroy(ev_end);
-        if (exec) cudaGraphExecDestroy(exec);
-        if (graph) cudaGraphDestroy(graph);
+        if (c->pend.exec) cudaGraphExecDestroy(c->pend.exec);
+        if (c->pend.graph) cudaGraphDestroy(c->pend.graph);
+        c->pend.exec = nullptr;
+        c->pend.graph = nullptr;
+        if (e2 != cudaSuccess) return fail(c, MPCGS_E_CUDA, std::string("sampling loop: ") + cudaGetErrorString(e2));
         c->loop_ms = ms;
     }
     if ((st = check_status(c))) return st;
-    c->nsamples = M;
-    c->lastN = N;
+    c->nsamples = c->pend.M;
+    c->lastN = c->pend.N;
     c->sample_theta0 = c->s.theta0;
     return MPCGS_OK;
 }
+}  // namespace
+
+extern "C" {
+
+mpcgs_status mpcgs_sample(mpcgs_ctx* c, int32_t N, int64_t M, uint64_t seed) {
+    mpcgs_status st = sample_begin(c, N, M, seed);
+    if (st) return st;
+    return sample_end(c);
+}
+
+mpcgs_status mpcgs_sample_loci(mpcgs_ctx* const* ctxs, int32_t n_loci, int32_t N, int64_t M,
+                               const uint64_t* seeds) {
+    if (!ctxs || !seeds || n_loci < 1) return MPCGS_E_ARG;
+    for (int32_t l = 0; l < n_loci; ++l)
+        if (!ctxs[l]) return MPCGS_E_ARG;
+    mpcgs_status first = MPCGS_OK;
+    int32_t begun = 0;
+    for (; begun < n_loci; ++begun) {  // enqueue every locus, then wait for all
+        mpcgs_status st = sample_begin(ctxs[begun], N, M, seeds[begun]);
+        if (st) { first = st; break; }
+    }
+    for (int32_t l = 0; l < begun; ++l) {
+        mpcgs_status st = sample_end(ctxs[l]);
+        if (st && !first) first = st;
+    }
+    return first;
+}
+
 
 mpcgs_status mpcgs_last_timing(const mpcgs_ctx* c, double* loop_ms, double* prune_ms, int64_t* launches) {
     if (!c) return MPCGS_E_ARG;
@@ -1363,29 +1427,54 @@ mpcgs_status mpcgs_log_rel_likelihood(mpcgs_ctx* c, double theta, double* out) {
     return MPCGS_OK;
 }
 
-mpcgs_status mpcgs_estimate_theta(mpcgs_ctx* c, double* theta_hat, int32_t G, double* grid_theta, double* grid_logL) {
-    CHECK_CTX(c);
-    if (c->nsamples < 1) return fail(c, MPCGS_E_STATE, "estimate_theta before sample");
-    if (!theta_hat || G < 3 || G > MPCGS_MAX_GRID) return fail(c, MPCGS_E_ARG, "n_grid must be in [3, 4096]");
-    mpcgs_status st = enter(c);
-    if (st) return st;
-    const int n = c->n;
-    double smin, smax;
-    if ((st = minmax(c, smin, smax))) return st;
-    if (smin == smax) {  // every stationary point is S/(n-1) (Appendix B)
-        *theta_hat = smin / (n - 1);
+}  // extern "C"
+
+namespace {
+// theta-hat of one or several loci sharing theta: the joint ln L
+// is the sum over loci of Eq. 25 (each locus with its own samples, n and theta0);
+// every stationary point solves sum_l S_w,l(theta) = theta sum_l (n_l - 1), so the
+// bracket is [sum_l S_min,l, sum_l S_max,l] / sum_l (n_l - 1) (S20).  One locus:
+// exactly the single-locus computation.
+mpcgs_status estimate_theta_impl(mpcgs_ctx* const* cs, int K, double* theta_hat, int32_t G, double* grid_theta,
+                                 double* grid_logL) {
+    mpcgs_ctx* c0 = cs[0];
+    for (int l = 0; l < K; ++l) {
+        CHECK_CTX(cs[l]);
+        if (cs[l]->nsamples < 1) return fail(cs[l], MPCGS_E_STATE, "estimate_theta before sample");
+        if (cs[l]->pend.active) return fail(cs[l], MPCGS_E_STATE, "a sampling loop is still pending");
+    }
+    if (!theta_hat || G < 3 || G > MPCGS_MAX_GRID) return fail(c0, MPCGS_E_ARG, "n_grid must be in [3, 4096]");
+    std::vector<double> smin(K), smax(K);
+    double smin_sum = 0.0, smax_sum = 0.0, dof = 0.0;
+    for (int l = 0; l < K; ++l) {
+        mpcgs_status st = enter(cs[l]);
+        if (st) return st;
+        if ((st = minmax(cs[l], smin[l], smax[l]))) return st;
+        smin_sum += smin[l];
+        smax_sum += smax[l];
+        dof += (double)(cs[l]->n - 1);
+    }
+    if (smin_sum == smax_sum) {  // every stationary point is S/(n-1) (Appendix B)
+        *theta_hat = smin_sum / dof;
         for (int g = 0; g < G; ++g) {
             if (grid_theta) grid_theta[g] = *theta_hat;
             if (grid_logL) grid_logL[g] = 0.0;
         }
         return MPCGS_OK;
     }
-    const double lo = smin / (n - 1), hi = smax / (n - 1);
-    double* buf = c->s.theta_buf;
-    CU(launch_theta_grid(c->s.sS, c->nsamples, n, c->sample_theta0, lo, hi, G, smin, smax, buf, c->work));
-    std::vector<double> h(2 * (size_t)G);
-    CU(cudaMemcpyAsync(h.data(), buf, 16 * (size_t)G, cudaMemcpyDeviceToHost, c->work));
-    CU(cudaStreamSynchronize(c->work));
+    const double lo = smin_sum / dof, hi = smax_sum / dof;
+    std::vector<double> h(2 * (size_t)G, 0.0), hl(2 * (size_t)G);
+    for (int l = 0; l < K; ++l) {  // ln L_l on the common grid, summed over loci
+        mpcgs_ctx* c = cs[l];
+        double* buf = c->s.theta_buf;
+        CU(launch_theta_grid(c->s.sS, c->nsamples, c->n, c->sample_theta0, lo, hi, G, smin[l], smax[l], buf, c->work));
+        CU(cudaMemcpyAsync(hl.data(), buf, 16 * (size_t)G, cudaMemcpyDeviceToHost, c->work));
+        CU(cudaStreamSynchronize(c->work));
+        for (int g = 0; g < G; ++g) {
+            h[g] = hl[g];
+            h[G + g] += hl[G + g];
+        }
+    }
     int best = 0;
     for (int g = 1; g < G; ++g)
         if (h[G + g] > h[G + best]) best = g;
@@ -1394,18 +1483,23 @@ mpcgs_status mpcgs_estimate_theta(mpcgs_ctx* c, double* theta_hat, int32_t G, do
     double blo = best > 0 ? h[best - 1] : lo, bhi = best < G - 1 ? h[best + 1] : hi;
     if (best == 0) blo = lo;
     if (best == G - 1) bhi = hi;
-    // f(theta) = S_w(theta) - (n-1) theta has the sign of d lnL / d theta
+    // f(theta) = sum_l (S_w,l - (n_l - 1) theta) has the sign of d lnL / d theta
     auto f_at = [&](double th, double& f, double& fp) -> mpcgs_status {
-        double m[4];
-        const double cen = (double)(n - 1) * th;
-        mpcgs_status s2 = moments(c, th, cen, smin, smax, m);
-        if (s2) return s2;
-        const double mean = m[1] / m[0];
-        f = mean;  // S_w - c with c = (n-1) theta
-        const double var = std::max(0.0, m[2] / m[0] - mean * mean);
-        fp = var / (th * th) - (double)(n - 1);
+        double fs = 0.0, vs = 0.0;
+        for (int l = 0; l < K; ++l) {
+            double m[4];
+            const double cen = (double)(cs[l]->n - 1) * th;
+            mpcgs_status s2 = moments(cs[l], th, cen, smin[l], smax[l], m);
+            if (s2) return s2;
+            const double mean = m[1] / m[0];
+            fs += mean;  // S_w - c with c = (n-1) theta
+            vs += std::max(0.0, m[2] / m[0] - mean * mean);
+        }
+        f = fs;
+        fp = vs / (th * th) - dof;
         return MPCGS_OK;
     };
+    mpcgs_status st;
     double flo, fhi, dummy;
     if ((st = f_at(blo, flo, dummy))) return st;
     if ((st = f_at(bhi, fhi, dummy))) return st;
@@ -1427,10 +1521,14 @@ mpcgs_status mpcgs_estimate_theta(mpcgs_ctx* c, double* theta_hat, int32_t G, do
     } else {
         // golden-section search on ln L inside the bracket
         auto ll = [&](double t, double& v) -> mpcgs_status {
-            double m[4];
-            mpcgs_status s2 = moments(c, t, 0.0, smin, smax, m);
-            if (s2) return s2;
-            v = (double)(n - 1) * std::log(c->sample_theta0 / t) + m[3] + std::log(m[0]);
+            double tot = 0.0;
+            for (int l = 0; l < K; ++l) {
+                double m[4];
+                mpcgs_status s2 = moments(cs[l], t, 0.0, smin[l], smax[l], m);
+                if (s2) return s2;
+                tot += (double)(cs[l]->n - 1) * std::log(cs[l]->sample_theta0 / t) + m[3] + std::log(m[0]);
+            }
+            v = tot;
             return MPCGS_OK;
         };
         const double gr = 0.6180339887498949;
@@ -1443,6 +1541,39 @@ mpcgs_status mpcgs_estimate_theta(mpcgs_ctx* c, double* theta_hat, int32_t G, do
         th = 0.5 * (a + bb);
     }
     *theta_hat = th;
+    return MPCGS_OK;
+}
+}  // namespace
+
+extern "C" {
+
+mpcgs_status mpcgs_estimate_theta(mpcgs_ctx* c, double* theta_hat, int32_t G, double* grid_theta, double* grid_logL) {
+    CHECK_CTX(c);
+    return estimate_theta_impl(&c, 1, theta_hat, G, grid_theta, grid_logL);
+}
+
+mpcgs_status mpcgs_estimate_theta_loci(mpcgs_ctx* const* ctxs, int32_t n_loci, double* theta_hat, int32_t G,
+                                       double* grid_theta, double* grid_logL) {
+    if (!ctxs || n_loci < 1) return MPCGS_E_ARG;
+    for (int32_t l = 0; l < n_loci; ++l)
+        if (!ctxs[l]) return MPCGS_E_ARG;
+    return estimate_theta_impl(ctxs, n_loci, theta_hat, G, grid_theta, grid_logL);
+}
+
+mpcgs_status mpcgs_em_loci(mpcgs_ctx* const* ctxs, int32_t n_loci, int32_t n_iter, int32_t N, int64_t M,
+                           const uint64_t* seeds, int32_t G, double* theta_trace) {
+    if (!ctxs || !seeds || n_loci < 1 || n_iter < 1 || M < 1) return MPCGS_E_ARG;
+    std::vector<uint64_t> sd(n_loci);
+    for (int32_t it = 0; it < n_iter; ++it) {
+        for (int32_t l = 0; l < n_loci; ++l) sd[l] = seeds[l] + (uint64_t)it;
+        mpcgs_status st = mpcgs_sample_loci(ctxs, n_loci, N, M, sd.data());
+        if (st) return st;
+        double th = 0.0;
+        if ((st = mpcgs_estimate_theta_loci(ctxs, n_loci, &th, G, nullptr, nullptr))) return st;
+        if (theta_trace) theta_trace[it] = th;
+        for (int32_t l = 0; l < n_loci; ++l)
+            if ((st = mpcgs_set_theta0(ctxs[l], th))) return st;
+    }
     return MPCGS_OK;
 }
 

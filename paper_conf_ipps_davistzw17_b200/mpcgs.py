@@ -77,6 +77,9 @@ _SIGS = {
     "mpcgs_set_theta0": (_i32, [_P, _f64]),
     "mpcgs_em": (_i32, [_P, _i32, _i32, _i64, _u64, _i32, _P]),
     "mpcgs_get_model": (_i32, [_P, _P, _P]),
+    "mpcgs_sample_loci": (_i32, [_P, _i32, _i32, _i64, _P]),
+    "mpcgs_estimate_theta_loci": (_i32, [_P, _i32, _P, _i32, _P, _P]),
+    "mpcgs_em_loci": (_i32, [_P, _i32, _i32, _i32, _i64, _P, _i32, _P]),
     "mpcgs_set_timing": (_i32, [_P, _i32]),
     "mpcgs_last_timing": (_i32, [_P, _P, _P, _P]),
     "mpcgs_last_error": (ctypes.c_char_p, [_P]),
@@ -199,6 +202,44 @@ def mpcgs_transition(model, kappa, pi, mu, t):
     if st:
         raise MpcgsError(st, "transition")
     return out.reshape(4, 4)
+
+
+# ------------------------------------------------------------------ multiple loci (f4)
+def _loci_args(contexts, seeds=None):
+    hs = (ctypes.c_void_p * len(contexts))(*[c.h for c in contexts])
+    sd = None if seeds is None else np.ascontiguousarray(seeds, np.uint64)
+    return hs, sd
+
+
+def _loci_err(st, contexts, what):
+    if st:
+        msgs = [lib().mpcgs_last_error(c.h).decode() for c in contexts if c.h]
+        raise MpcgsError(st, f"{what}: {'; '.join(m for m in msgs if m)}")
+
+
+def mpcgs_sample_loci(contexts, n_proposals, n_samples, seeds):
+    """Sample every locus (one Context each) with its own seed; loops overlap on the GPU."""
+    hs, sd = _loci_args(contexts, seeds)
+    _loci_err(lib().mpcgs_sample_loci(hs, len(contexts), n_proposals, n_samples, _ptr(sd)), contexts,
+              "sample_loci")
+
+
+def mpcgs_estimate_theta_loci(contexts, n_grid=256, curve=False):
+    """Joint theta-hat of loci sharing theta (product of Eq. 25 over loci)."""
+    hs, _ = _loci_args(contexts)
+    th = ctypes.c_double()
+    gt, gl = np.zeros(n_grid), np.zeros(n_grid)
+    _loci_err(lib().mpcgs_estimate_theta_loci(hs, len(contexts), ctypes.byref(th), n_grid, _ptr(gt), _ptr(gl)),
+              contexts, "estimate_theta_loci")
+    return (th.value, gt, gl) if curve else th.value
+
+
+def mpcgs_em_loci(contexts, n_iter, n_proposals, n_samples, seeds, n_grid=256):
+    hs, sd = _loci_args(contexts, seeds)
+    trace = np.zeros(n_iter)
+    _loci_err(lib().mpcgs_em_loci(hs, len(contexts), n_iter, n_proposals, n_samples, _ptr(sd), n_grid,
+                                  _ptr(trace)), contexts, "em_loci")
+    return trace
 
 
 def mpcgs_nccl_unique_id():
