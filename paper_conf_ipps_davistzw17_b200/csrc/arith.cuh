@@ -93,6 +93,18 @@ __device__ __forceinline__ void ld4<float>(float (&r)[4], const float* p) {
 }
 
 template <typename T>
+__device__ __forceinline__ void st4(T* p, const T (&r)[4]);
+template <>
+__device__ __forceinline__ void st4<double>(double* p, const double (&r)[4]) {
+    reinterpret_cast<double2*>(p)[0] = make_double2(r[0], r[1]);
+    reinterpret_cast<double2*>(p)[1] = make_double2(r[2], r[3]);
+}
+template <>
+__device__ __forceinline__ void st4<float>(float* p, const float (&r)[4]) {
+    *reinterpret_cast<float4*>(p) = make_float4(r[0], r[1], r[2], r[3]);
+}
+
+template <typename T>
 __device__ __forceinline__ T pick4(const T (&v)[4], int x) {
     return x == 0 ? v[0] : (x == 1 ? v[1] : (x == 2 ? v[2] : v[3]));
 }

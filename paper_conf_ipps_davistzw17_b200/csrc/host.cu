@@ -446,14 +446,18 @@ void upgma(int n, int L, const uint8_t* codes, double theta0, int32_t* parent, d
     }
 }
 
-// Sites per CTA: a multiple of the kernel's site batch, as many batches as keep
+// Sites per CTA: a multiple of the kernel's site batch (up to 16 batches: amortises the
+// per-CTA table setup), as many batches as keep
 // >= ~8 CTAs per SM busy.  Depends only on L and the GLOBAL tree count, so every
 // rank tiles (and sums) a proposal's sites identically (world-size invariance).
+#ifndef MPCGS_MAXPER
+#define MPCGS_MAXPER 16
+#endif
 void prune_tiling(int n, int L, int ntrees_global, int precision, int& tiles, int& sites_per_cta) {
     const int batch = prune_batch_sites(n, precision);
     const long batches = (L + batch - 1) / batch;
     const long want = (long)148 * 8;
-    const int per = (int)std::max<long>(1, std::min<long>(8, (ntrees_global * batches) / want));
+    const int per = (int)std::max<long>(1, std::min<long>(MPCGS_MAXPER, (ntrees_global * batches) / want));
     sites_per_cta = per * batch;
     tiles = (L + sites_per_cta - 1) / sites_per_cta;
 }

@@ -35,6 +35,7 @@ struct PruneArgs {
     const double* site_w;      // [L] pattern counts (compressed sites, f3) or nullptr
     const int32_t* tree_need;  // [ntrees] register need of each tree's schedule (nullable)
     int need_cap;              // set by launch_prune: largest need the table kernel serves
+    int trip_cap;              // set by launch_prune: fused triplets per tree (table kernel)
     double* tile_part;         // [ntrees][tiles]
     uint32_t* tile_cnt;        // [ntrees], zero on entry, reset by the kernel
     double* out;               // logL of tree t -> out[(out_first + t) * out_stride]

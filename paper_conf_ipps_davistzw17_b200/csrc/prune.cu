@@ -30,15 +30,20 @@ int prune_batch_sites(int n, int precision) { return PRUNE_THREADS * prune_si(n,
 
 // register need the table kernel serves (DR registers + PRUNE_SPILL shared levels);
 // deeper trees (rare) are scored by the flat kernel in a second pass
-int prune_need_cap(int n) { return std::min(prune_max_need(n), PRUNE_DR + PRUNE_SPILL); }
+// One shared spill level up to n = 64 (a random coalescent tree of 64 tips needs
+// more than DR + 1 = 4 registers about once in 140), two above.
+#ifndef MPCGS_SPILL64
+#define MPCGS_SPILL64 1
+#endif
+int prune_need_cap(int n) { return std::min(prune_max_need(n), PRUNE_DR + (n <= 64 ? MPCGS_SPILL64 : PRUNE_SPILL)); }
 
 
 template <typename T, bool GM>
 static size_t tab_bytes_for(int n) {
     const int cap = prune_need_cap(n);
     constexpr int SI = sizeof(T) == 4 ? PRUNE_SI32 : PRUNE_SI64;
-    return product_tables(n) ? tab_smem_bytes<T, PRUNE_DR, SI, true, GM>(n - 1, cap)
-                             : tab_smem_bytes<T, PRUNE_DR, PRUNE_SI_LARGE, false, GM>(n - 1, cap);
+    return product_tables(n) ? tab_smem_bytes<T, PRUNE_DR, SI, true, GM>(n - 1, cap, 0)
+                             : tab_smem_bytes<T, PRUNE_DR, PRUNE_SI_LARGE, false, GM>(n - 1, cap, 0);
 }
 
 bool prune_uses_tables(int n, int precision, bool general_model) {

@@ -370,6 +370,102 @@ struct Codes {
 
 constexpr uint32_t TAB_CHECK = 0x80000000u;  // toff flag: the cherry table can hold small vectors
 
+// Sparse underflow checks (S5).  Every component of a branch-transformed child
+// vector is >= d(child) * max(child), d = em * pi_min under F81 (Eq. 20: P_XY >=
+// em pi_Y) or min_XY P_XY(t) under a general model, and a tip is a one-hot
+// vector (max 1).  A node's vector is the product of its two transformed
+// children, so log2 of its smallest component is bounded below by the sum of its
+// children's bounds and ilogb(d_a) + ilogb(d_b).  mark_checks walks the schedule
+// once per CTA with these integer bounds and sets OP_CHECK only on the ops whose
+// result could otherwise come within reach of underflow; the check itself is
+// unchanged (rescale by an exact power of two when max < 2^-TS), so the result
+// is bit-identical to checking every node.
+#ifndef MPCGS_SPARSE
+#define MPCGS_SPARSE 1
+#endif
+#ifndef MPCGS_NO_TRIPLETS
+#define MPCGS_NO_TRIPLETS 0
+#endif
+constexpr uint32_t OP_CHECK = 1u << 28;  // op code flag (bits 28-31 are free): check this op's result
+// Fused triplet (table kernel only): a cherry (TT, tips a and b) immediately
+// followed by the TS op that joins it to tip c -- one 64x4 table of the result
+// over (x_a, x_b, x_c), built per CTA.  Type 3 is unused by the schedule encoding.
+constexpr uint32_t OP_TTT = 3u;
+constexpr int TRIP_EXTRA = 256 - 64 - 16;  // table values a fused triplet adds (64x4 vs 16x4 + 4x4)
+constexpr int BOUND_NEG_INF = -100000;   // ilogb of 0 (or of a subnormal): no bound
+// FP64 only: FP32's range leaves no room between checks (every op would be flagged)
+template <typename T>
+__host__ __device__ constexpr bool sparse_checks() { return MPCGS_SPARSE && sizeof(T) == 8; }
+
+template <typename T>
+struct Bounds;
+template <>
+struct Bounds<double> {
+    static constexpr int FLOOR = -1000;  // keep every component >= 2^-1000 (normal, 22 bits of margin)
+    __device__ static int ilogb(double x) {
+        const int ex = (__double2hiint(x) >> 20) & 2047;
+        return (x > 0.0 && ex > 0) ? ex - 1023 : BOUND_NEG_INF;
+    }
+};
+template <>
+struct Bounds<float> {
+    static constexpr int FLOOR = -120;
+    __device__ static int ilogb(float x) {
+        const int ex = (__float_as_int(x) >> 23) & 255;
+        return (x > 0.0f && ex > 0) ? ex - 127 : BOUND_NEG_INF;
+    }
+};
+
+// One thread: s_d[2 op + c] = lower bound of log2 d of child c of original op
+// `op`; lpmin = ilogb(min pi) (the root's Eq. 21 dot product).  Walks the
+// compacted op list s_opc (a fused triplet, type OP_TTT, covers original ops o
+// and o+1) and sets s_chk[i] for the ops to check (merged into OP_CHECK later).
+// compacted op record of the table kernel: {code, table byte offset, original op
+// index, tip c of a fused triplet} and the op's F81 branch data (one address, so
+// the two loads of an op do not depend on each other)
+template <typename T>
+struct __align__(16) OpRec {
+    uint4 h;
+    typename Traits<T>::E4 ed;
+};
+
+template <typename T>
+__device__ void mark_checks(const OpRec<T>* s_opc, const int* s_d, int* s_bnd, unsigned char* s_chk, int nops_c,
+                            int lpmin) {
+    constexpr int TSX = Traits<T>::TS, FLOOR = Bounds<T>::FLOOR;
+    auto dsum = [&](const uint4& o) {
+        const int i = (int)o.z;
+        int d = s_d[2 * i] + s_d[2 * i + 1];
+        if ((o.x & 3u) == OP_TTT) d += s_d[2 * i + 2] + s_d[2 * i + 3];
+        return d;
+    };
+    int dmax = 0;
+    for (int i = 0; i < nops_c; ++i) dmax = max(dmax, -dsum(s_opc[i].h));
+    // stack entries stay >= limit, so an op's product is >= 2 limit - dmax >= FLOOR
+    const int x = FLOOR + dmax;
+    const int limit = x >= 0 ? (x + 1) / 2 : -((-x) / 2);
+    const bool all = limit > -TSX;  // no room between checks (e.g. a zero-length branch): check every op
+    for (int i = 0; i < nops_c; ++i) {
+        const uint4 o = s_opc[i].h;
+        const int ty = (int)(o.x & 3u), sp = (int)((o.x >> 2) & 15u);
+        int b = dsum(o), slot;
+        if (ty == (int)OP_TT || ty == (int)OP_TTT) {
+            slot = sp;
+        } else if (ty == (int)OP_TS) {
+            slot = sp - 1;
+            b += s_bnd[sp - 1];
+        } else {
+            slot = sp - 2;
+            b += s_bnd[sp - 2] + s_bnd[sp - 1];
+        }
+        const bool chk = all || b < limit || (i == nops_c - 1 && b + lpmin < FLOOR);
+        if (chk) b = -TSX;  // after the check: max >= 2^-TS
+        s_chk[i] = chk;
+        s_bnd[slot] = b;
+    }
+}
+
+
 template <typename T, int DR, int SI, bool PT, int S, int DMX>
 __device__ __forceinline__ void tab_tt(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, const T* s_tab,
                                        const Codes<SI>& c, int (&scale)[SI]) {
@@ -383,7 +479,7 @@ __device__ __forceinline__ void tab_tt(Stack<T, DR, SI>& st, uint32_t code, uint
 #pragma unroll
             for (int k = 0; k < SI; ++k)
                 ld4<T>(v[k], reinterpret_cast<const T*>(base + c.template off4<EB>(wa, k) + c.template off<EB>(wb, k)));
-            if (toff & TAB_CHECK) rescale_sites<T, SI>(v, scale);
+            if (sparse_checks<T>() ? (code & OP_CHECK) != 0u : (toff & TAB_CHECK) != 0u) rescale_sites<T, SI>(v, scale);
         } else {             // two 4x4 tip tables, multiplied here
 #pragma unroll
             for (int k = 0; k < SI; ++k) {
@@ -393,8 +489,29 @@ __device__ __forceinline__ void tab_tt(Stack<T, DR, SI>& st, uint32_t code, uint
 #pragma unroll
                 for (int i = 0; i < 4; ++i) v[k][i] *= w[i];
             }
-            rescale_sites<T, SI>(v, scale);
+            if (!sparse_checks<T>() || (code & OP_CHECK)) rescale_sites<T, SI>(v, scale);
         }
+#pragma unroll
+        for (int k = 0; k < SI; ++k) st.template put<S>(k, v[k]);
+    }
+}
+
+// fused triplet: one lookup in the 64x4 table of tip(c) (.) branch(tip(a) (.) tip(b))
+template <typename T, int DR, int SI, bool PT, int S, int DMX>
+__device__ __forceinline__ void tab_ttt(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, uint32_t tc,
+                                        const T* s_tab, const Codes<SI>& c, int (&scale)[SI]) {
+    if constexpr (PT && S < DMX) {
+        constexpr int EB = 4 * sizeof(T);
+        const uint32_t wa = c.word((code >> 6) & 2047);
+        const uint32_t wb = c.word((code >> 17) & 2047);
+        const uint32_t wc = c.word((int)tc);
+        const char* base = reinterpret_cast<const char*>(s_tab) + (toff & ~TAB_CHECK);
+        T v[SI][4];
+#pragma unroll
+        for (int k = 0; k < SI; ++k)
+            ld4<T>(v[k], reinterpret_cast<const T*>(base + (c.template off4<EB>(wa, k) << 2) +
+                                                    c.template off4<EB>(wb, k) + c.template off<EB>(wc, k)));
+        if (sparse_checks<T>() ? (code & OP_CHECK) != 0u : (toff & TAB_CHECK) != 0u) rescale_sites<T, SI>(v, scale);
 #pragma unroll
         for (int k = 0; k < SI; ++k) st.template put<S>(k, v[k]);
     }
@@ -405,12 +522,24 @@ __device__ __forceinline__ void tab_tt(Stack<T, DR, SI>& st, uint32_t code, uint
 template <typename T, bool GM>
 using BranchData = std::conditional_t<GM, const T*, typename Traits<T>::E4>;
 
+// the branch data of one child, loaded once per op (outside the per-site loop)
 template <typename T, bool GM, bool SECOND>
-__device__ __forceinline__ void branch_op(T (&v)[4], const BranchData<T, GM>& bd, const T (&pi)[4]) {
-    if constexpr (GM) gm_branch<T>(v, bd + (SECOND ? 16 : 0));
-    else if constexpr (SECOND) branch<T>(v, bd.z, bd.w, pi);
-    else branch<T>(v, bd.x, bd.y, pi);
-}
+struct ChildBr {
+    std::conditional_t<GM, const T*, T> e;
+    T em;
+    __device__ __forceinline__ ChildBr(const BranchData<T, GM>& bd) {
+        if constexpr (GM) {
+            e = bd + (SECOND ? 16 : 0);
+        } else {
+            e = SECOND ? bd.z : bd.x;
+            em = SECOND ? bd.w : bd.y;
+        }
+    }
+    __device__ __forceinline__ void apply(T (&v)[4], const T (&pi)[4]) const {
+        if constexpr (GM) gm_branch<T>(v, e);
+        else branch<T>(v, e, em, pi);
+    }
+};
 
 template <typename T, int DR, int SI, int S, int DMX, bool GM>
 __device__ __forceinline__ void tab_ts(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff,
@@ -420,47 +549,51 @@ __device__ __forceinline__ void tab_ts(Stack<T, DR, SI>& st, uint32_t code, uint
         constexpr int EB = 4 * sizeof(T);
         const uint32_t wa = c.word((code >> 6) & 2047);
         const char* base = reinterpret_cast<const char*>(s_tab) + toff;
+        const ChildBr<T, GM, true> cb(ed);
         T v[SI][4];
 #pragma unroll
         for (int k = 0; k < SI; ++k) {
             T tip[4];
             ld4<T>(tip, reinterpret_cast<const T*>(base + c.template off<EB>(wa, k)));
             st.template get<S - 1>(k, v[k]);
-            branch_op<T, GM, true>(v[k], ed, pi);
+            cb.apply(v[k], pi);
 #pragma unroll
             for (int i = 0; i < 4; ++i) v[k][i] *= tip[i];
         }
-        rescale_sites<T, SI>(v, scale);
+        if (!sparse_checks<T>() || (code & OP_CHECK)) rescale_sites<T, SI>(v, scale);
 #pragma unroll
         for (int k = 0; k < SI; ++k) st.template put<S - 1>(k, v[k]);
     }
 }
 
 template <typename T, int DR, int SI, int S, int DMX, bool GM>
-__device__ __forceinline__ void tab_ss(Stack<T, DR, SI>& st, const BranchData<T, GM>& ed, const T (&pi)[4],
-                                       int (&scale)[SI]) {
+__device__ __forceinline__ void tab_ss(Stack<T, DR, SI>& st, uint32_t code, const BranchData<T, GM>& ed,
+                                       const T (&pi)[4], int (&scale)[SI]) {
     if constexpr (S >= 2 && S <= DMX) {
+        const ChildBr<T, GM, false> ca(ed);
+        const ChildBr<T, GM, true> cb(ed);
         T v[SI][4];
 #pragma unroll
         for (int k = 0; k < SI; ++k) {
             T w[4];
             st.template get<S - 2>(k, v[k]);
             st.template get<S - 1>(k, w);
-            branch_op<T, GM, false>(v[k], ed, pi);
-            branch_op<T, GM, true>(w, ed, pi);
+            ca.apply(v[k], pi);
+            cb.apply(w, pi);
 #pragma unroll
             for (int i = 0; i < 4; ++i) v[k][i] *= w[i];
         }
-        rescale_sites<T, SI>(v, scale);
+        if (!sparse_checks<T>() || (code & OP_CHECK)) rescale_sites<T, SI>(v, scale);
 #pragma unroll
         for (int k = 0; k < SI; ++k) st.template put<S - 2>(k, v[k]);
     }
 }
 
 #define MPCGS_TABCASE(S)                                                                          \
-    case 3 * (S) + 0: tab_tt<T, DR, SI, PT, S, DMX>(st, code, toff, s_tab, cc, scale); break;       \
-    case 3 * (S) + 1: tab_ts<T, DR, SI, S, DMX, GM>(st, code, toff, ed, s_tab, cc, pi, scale); break; \
-    case 3 * (S) + 2: tab_ss<T, DR, SI, S, DMX, GM>(st, ed, pi, scale); break;
+    case 4 * (S) + 0: tab_tt<T, DR, SI, PT, S, DMX>(st, code, toff, s_tab, cc, scale); break;       \
+    case 4 * (S) + 1: tab_ts<T, DR, SI, S, DMX, GM>(st, code, toff, ed, s_tab, cc, pi, scale); break; \
+    case 4 * (S) + 2: tab_ss<T, DR, SI, S, DMX, GM>(st, code, ed, pi, scale); break;                  \
+    case 4 * (S) + 3: tab_ttt<T, DR, SI, PT, S, DMX>(st, code, toff, tc, s_tab, cc, scale); break;
 #define MPCGS_CASES_4 MPCGS_TABCASE(0) MPCGS_TABCASE(1) MPCGS_TABCASE(2) MPCGS_TABCASE(3) MPCGS_TABCASE(4)
 #define MPCGS_CASES_6 MPCGS_CASES_4 MPCGS_TABCASE(5) MPCGS_TABCASE(6)
 #define MPCGS_CASES_8 MPCGS_CASES_6 MPCGS_TABCASE(7) MPCGS_TABCASE(8)
@@ -468,7 +601,7 @@ __device__ __forceinline__ void tab_ss(Stack<T, DR, SI>& st, const BranchData<T,
 
 // one op for SI sites; the switch only has the (sp, type) labels a DMX-level tree can use
 template <typename T, int DR, int SI, bool PT, int DMX, bool GM>
-__device__ __forceinline__ void run_op(int di, Stack<T, DR, SI>& st, uint32_t code, uint32_t toff,
+__device__ __forceinline__ void run_op(int di, Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, uint32_t tc,
                                        const BranchData<T, GM>& ed, const T* s_tab, const Codes<SI>& cc,
                                        const T (&pi)[4], int (&scale)[SI]) {
     if constexpr (DMX <= 4) {
@@ -485,14 +618,16 @@ __device__ __forceinline__ void run_op(int di, Stack<T, DR, SI>& st, uint32_t co
 __host__ __device__ constexpr size_t align16(size_t x) { return (x + 15) & ~(size_t)15; }
 
 // shared memory of the table kernel for trees of n tips whose register need is
-// at most `need` (spill levels above DR)
+// at most `need` (spill levels above DR), with up to `trip_cap` fused triplets
 template <typename T, int DR, int SI, bool PT, bool GM = false>
-__host__ __device__ size_t tab_smem_bytes(int nops, int need) {
+__host__ __device__ size_t tab_smem_bytes(int nops, int need, int trip_cap) {
     const int n = nops + 1;
     const int spill = need > DR ? need - DR : 0;
-    return align16((GM ? 32 * sizeof(T) : sizeof(typename Traits<T>::E4)) * nops) + align16(sizeof(T) * (PT ? 32 : 16) * (size_t)n) +
-           align16(sizeof(uint2) * nops) + 2 * align16(Codes<SI>::buf_bytes(n)) +
-           sizeof(T) * (size_t)spill * SI * 4 * PRUNE_THREADS;
+    return align16((GM ? 32 * sizeof(T) : sizeof(typename Traits<T>::E4)) * nops) +
+           align16(sizeof(T) * ((PT ? 32 : 16) * (size_t)n + (size_t)TRIP_EXTRA * (PT ? trip_cap : 0))) +
+           align16(sizeof(OpRec<T>) * nops) + 2 * align16(Codes<SI>::buf_bytes(n)) +
+           sizeof(T) * (size_t)spill * SI * 4 * PRUNE_THREADS +
+           align16(sizeof(int) * 2 * (size_t)nops) + align16(sizeof(int) * (size_t)nops) + 64 * sizeof(int);
 }
 
 #ifdef MPCGS_MINB  // tuning builds only: min CTAs per SM (caps registers)
@@ -509,15 +644,24 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
     constexpr size_t OPB = GM ? 32 * sizeof(T) : sizeof(E4);  // branch data bytes per op
     extern __shared__ __align__(16) unsigned char smem_raw[];
     const int nops = a.nops, n = nops + 1;
+    const int trip_cap = PT ? a.trip_cap : 0;
     E4* s_e = reinterpret_cast<E4*>(smem_raw);  // F81: {e_a, em_a, e_b, em_b} per op
     T* s_P = reinterpret_cast<T*>(smem_raw);    // general model: {P_a, P_b} per op
     T* s_tab = reinterpret_cast<T*>(smem_raw + align16(OPB * nops));
-    uint2* s_op = reinterpret_cast<uint2*>(reinterpret_cast<unsigned char*>(s_tab) + align16(sizeof(T) * TABE * n));
-    unsigned char* s_cod = reinterpret_cast<unsigned char*>(s_op) + align16(sizeof(uint2) * nops);
+    // compacted ops: {code, table byte offset, original op index, tip c of a fused triplet}
+    OpRec<T>* s_opc = reinterpret_cast<OpRec<T>*>(reinterpret_cast<unsigned char*>(s_tab) +
+                                            align16(sizeof(T) * (TABE * n + (size_t)TRIP_EXTRA * trip_cap)));
+    unsigned char* s_cod = reinterpret_cast<unsigned char*>(s_opc) + align16(sizeof(OpRec<T>) * nops);
     const size_t bufb = align16(CD::buf_bytes(n));
     T* s_spill = reinterpret_cast<T*>(s_cod + 2 * bufb);
+    const int spill_lv = a.need_cap > DR ? a.need_cap - DR : 0;
+    int* s_d = reinterpret_cast<int*>(reinterpret_cast<unsigned char*>(s_spill) +
+                                      sizeof(T) * (size_t)spill_lv * SI * 4 * PRUNE_THREADS);
+    int* s_tl = s_d + align16(sizeof(int) * 2 * (size_t)nops) / sizeof(int);  // original codes, then check flags
+    int* s_bnd = s_tl + align16(sizeof(int) * (size_t)nops) / sizeof(int);
     __shared__ double s_red[PRUNE_THREADS / 32];
     __shared__ bool s_last;
+    __shared__ int s_nc;  // compacted op count
 
     const int tid = threadIdx.x;
     const int tree = blockIdx.y;
@@ -540,91 +684,181 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
     };
     if (nb > 0) issue(0, 0);
 
-    // schedule, then per-op table byte offsets (warp 0 scan), then the tables
+    // 1. schedule, branch data and the per-child bounds d (mark_checks, fusion guard)
     const uint32_t* __restrict__ gop = a.sched_op + (size_t)tree * nops;
     const E4* __restrict__ ge = reinterpret_cast<const E4*>(a.sched_e) + (size_t)tree * nops;
+    const T pi[4] = {(T)a.pi[0], (T)a.pi[1], (T)a.pi[2], (T)a.pi[3]};
+    const T pimin = min(min(pi[0], pi[1]), min(pi[2], pi[3]));
+    uint32_t* s_code = reinterpret_cast<uint32_t*>(s_tl);  // original codes (s_tl is filled after the scan)
     for (int i = tid; i < nops; i += PRUNE_THREADS) {
-        s_op[i].x = gop[i];
-        if constexpr (!GM) s_e[i] = ge[i];
+        s_code[i] = gop[i];
+        if constexpr (!GM) {  // d = em pi_min (Eq. 20)
+            const E4 ed = ge[i];
+            s_e[i] = ed;
+            const int lp = Bounds<T>::ilogb(pimin);
+            s_d[2 * i] = Bounds<T>::ilogb((T)ed.y) + lp;
+            s_d[2 * i + 1] = Bounds<T>::ilogb((T)ed.w) + lp;
+        }
     }
-    if constexpr (GM) {  // {P_a, P_b} of every op from its branch lengths {t_a, 0, t_b, 0}
+    if constexpr (GM) {  // {P_a, P_b} of every op from its branch lengths {t_a, 0, t_b, 0}; d = min_XY P_XY(t)
         for (int i = tid; i < nops * 2; i += PRUNE_THREADS) {
             const E4 ed = ge[i >> 1];
             double P[16];
             pmat(a.gm, (double)((i & 1) ? ed.z : ed.x), P);
+            T pmin = (T)P[0];
 #pragma unroll
-            for (int k = 0; k < 16; ++k) s_P[i * 16 + k] = (T)P[k];
+            for (int k = 0; k < 16; ++k) {
+                s_P[i * 16 + k] = (T)P[k];
+                pmin = min(pmin, (T)P[k]);
+            }
+            s_d[i] = Bounds<T>::ilogb(pmin);
         }
     }
     __syncthreads();
+    // 2. warp 0: fuse the first trip_cap (TT, TS) pairs, compact the op list and
+    //    lay out the tables (exclusive scans over the original ops)
     if (tid < 32) {
-        uint32_t carry = 0;
+        uint32_t c_keep = 0, c_size = 0, c_cand = 0, prev_start = 0;
         for (int base = 0; base < nops; base += 32) {
             const int i = base + tid;
-            uint32_t sz = 0;
+            uint32_t code = 0, ty = 2, tyn = 2;
             if (i < nops) {
-                const uint32_t ty = s_op[i].x & 3u;
-                sz = ty == OP_TT ? 2u * TABE : (ty == OP_TS ? 16u : 0u);
+                code = s_code[i];
+                ty = code & 3u;
+                if (i + 1 < nops) tyn = s_code[i + 1] & 3u;
             }
+            // candidate: a cherry whose parent joins it to a tip, with table values safely normal
+            const bool cand = PT && i < nops && ty == OP_TT && tyn == OP_TS &&
+                              s_d[2 * i] + s_d[2 * i + 1] + s_d[2 * i + 2] + s_d[2 * i + 3] >= Bounds<T>::FLOOR / 2;
+            const unsigned mc = __ballot_sync(0xffffffffu, cand);
+            const uint32_t rank = c_cand + __popc(mc & ((1u << tid) - 1u));
+            const bool start = cand && rank < (uint32_t)trip_cap;
+            const unsigned ms = __ballot_sync(0xffffffffu, start);
+            const bool prev = tid == 0 ? prev_start != 0u : ((ms >> (tid - 1)) & 1u) != 0u;
+            const bool keep = i < nops && !(ty == OP_TS && prev);
+            uint32_t sz = 0;
+            if (keep) sz = start ? 256u : (ty == OP_TT ? 2u * TABE : (ty == OP_TS ? 16u : 0u));
+            const unsigned mk = __ballot_sync(0xffffffffu, keep);
+            const uint32_t j = c_keep + __popc(mk & ((1u << tid) - 1u));
             uint32_t x = sz;
 #pragma unroll
             for (int o = 1; o < 32; o <<= 1) {
                 const uint32_t y = __shfl_up_sync(0xffffffffu, x, o);
                 if (tid >= o) x += y;
             }
-            if (i < nops) s_op[i].y = (carry + x - sz) * (uint32_t)sizeof(T);  // byte offset
-            carry += __shfl_sync(0xffffffffu, x, 31);
-        }
-    }
-    __syncthreads();
-    const T pi[4] = {(T)a.pi[0], (T)a.pi[1], (T)a.pi[2], (T)a.pi[3]};
-    for (int idx = tid; idx < nops * 64; idx += PRUNE_THREADS) {
-        const int op = idx >> 6, j = idx & 63;
-        const uint32_t ty = s_op[op].x & 3u;
-        T* tab = reinterpret_cast<T*>(reinterpret_cast<char*>(s_tab) + s_op[op].y);
-        if constexpr (GM) {  // entries are columns of P_a / P_b (row X = parent state)
-            const T* Pa = s_P + op * 32;
-            const T* Pb = Pa + 16;
-            if (ty == OP_TT && PT) {
-                const int xa = j >> 4, xb = (j >> 2) & 3, X = j & 3;
-                tab[j] = Pa[X * 4 + xa] * Pb[X * 4 + xb];
-            } else if (ty == OP_TT && j < 32) {
-                const int x = (j >> 2) & 3, X = j & 3;
-                tab[j] = j < 16 ? Pa[X * 4 + x] : Pb[X * 4 + x];
-            } else if (ty == OP_TS && j < 16) {
-                const int x = j >> 2, X = j & 3;
-                tab[j] = Pa[X * 4 + x];
+            const uint32_t tc = (i + 1 < nops) ? ((s_code[i + 1] >> 6) & 2047u) : 0u;
+            __syncwarp();
+            if (keep) {
+                const uint32_t cx = start ? ((code & ~3u) | OP_TTT) : code;
+                s_opc[j].h = make_uint4(cx, (c_size + x - sz) * (uint32_t)sizeof(T), (uint32_t)i, start ? tc : 0u);
+                if constexpr (!GM) s_opc[j].ed = s_e[i];
             }
-            continue;
+            c_size += __shfl_sync(0xffffffffu, x, 31);
+            c_keep += __popc(mk);
+            c_cand += __popc(mc);
+            prev_start = (ms >> 31) & 1u;
         }
-        const E4 ed = s_e[op];
-        if (ty == OP_TT && PT) {
-            // cherry: entry (xa, xb) = P_{.,xa}(t_a) (.) P_{.,xb}(t_b)   (Eq. 19-20 at two tips)
-            const int xa = j >> 4, xb = (j >> 2) & 3, X = j & 3;
-            const T va = (X == xa ? (T)ed.x : T(0)) + (T)ed.y * pick4(pi, xa);
-            const T vb = (X == xb ? (T)ed.z : T(0)) + (T)ed.w * pick4(pi, xb);
-            tab[j] = va * vb;
-        } else if (ty == OP_TT && j < 32) {  // two tip tables: a at [0, 16), b at [16, 32)
-            const int x = (j >> 2) & 3, X = j & 3;
-            tab[j] = j < 16 ? (X == x ? (T)ed.x : T(0)) + (T)ed.y * pick4(pi, x)
-                            : (X == x ? (T)ed.z : T(0)) + (T)ed.w * pick4(pi, x);
-        } else if (ty == OP_TS && j < 16) {
-            const int x = j >> 2, X = j & 3;
-            tab[j] = (X == x ? (T)ed.x : T(0)) + (T)ed.y * pick4(pi, x);
+        if (tid == 0) s_nc = (int)c_keep;
+    }
+    __syncthreads();
+    const int nops_c = s_nc;
+    // 3. sparse checks (FP64): one thread walks the bounds while the others build the tables
+    unsigned char* s_chk = reinterpret_cast<unsigned char*>(s_tl);  // s_code is dead after the scan
+    if constexpr (sparse_checks<T>()) {
+        if (tid == 32) mark_checks<T>(s_opc, s_d, s_bnd, s_chk, nops_c, Bounds<T>::ilogb(pimin));
+    }
+    //    tables, one 4-vector (row) per work item: tip tables P_{.,x}(t) (Eq. 19-20 at an
+    //    indicator tip), cherry rows tip_a(xa) (.) tip_b(xb), and fused-triplet rows
+    //    tip_c(xc) (.) branch(tip_a(xa) (.) tip_b(xb)) for the four xc -- the TS op
+    //    applied to the cherry's vector, as the per-site path computes it
+    for (int idx = tid; idx < nops_c * 16; idx += PRUNE_THREADS) {
+        const int op = idx >> 4, r = idx & 15;
+        const uint4 ox = s_opc[op].h;
+        const uint32_t ty = ox.x & 3u;
+        T* tab = reinterpret_cast<T*>(reinterpret_cast<char*>(s_tab) + (ox.y & ~TAB_CHECK));
+        T va[4], vb[4];
+        if constexpr (GM) {  // tip vectors are columns of P (row X = parent state)
+            const T* Pa = s_P + ox.z * 32;
+            auto col = [](T (&v)[4], const T* P, int x) {
+#pragma unroll
+                for (int X = 0; X < 4; ++X) v[X] = P[X * 4 + x];
+            };
+            if (ty == OP_TT && PT) {
+                col(va, Pa, r >> 2);
+                col(vb, Pa + 16, r & 3);
+#pragma unroll
+                for (int X = 0; X < 4; ++X) va[X] *= vb[X];
+                st4<T>(tab + r * 4, va);
+            } else if (ty == OP_TT && r < 8) {
+                col(va, Pa + (r < 4 ? 0 : 16), r & 3);
+                st4<T>(tab + r * 4, va);
+            } else if (ty == OP_TS && r < 4) {
+                col(va, Pa, r);
+                st4<T>(tab + r * 4, va);
+            } else if (ty == OP_TTT) {  // op o: P_a, P_b; op o+1: P of tip c, P of the cherry's branch
+                const T* Pc = Pa + 32;
+                col(va, Pa, r >> 2);
+                col(vb, Pa + 16, r & 3);
+#pragma unroll
+                for (int X = 0; X < 4; ++X) va[X] *= vb[X];
+                gm_branch<T>(va, Pc + 16);
+#pragma unroll
+                for (int xc = 0; xc < 4; ++xc) {
+                    col(vb, Pc, xc);
+#pragma unroll
+                    for (int X = 0; X < 4; ++X) vb[X] *= va[X];
+                    st4<T>(tab + (r * 4 + xc) * 4, vb);
+                }
+            }
+        } else {
+            const E4 ed = s_e[ox.z];
+            if (ty == OP_TT && PT) {
+                tipvec<T>(va, r >> 2, (T)ed.x, (T)ed.y, pi);
+                tipvec<T>(vb, r & 3, (T)ed.z, (T)ed.w, pi);
+#pragma unroll
+                for (int X = 0; X < 4; ++X) va[X] *= vb[X];
+                st4<T>(tab + r * 4, va);
+            } else if (ty == OP_TT && r < 8) {  // two tip tables: a at [0, 16), b at [16, 32)
+                if (r < 4) tipvec<T>(va, r, (T)ed.x, (T)ed.y, pi);
+                else tipvec<T>(va, r - 4, (T)ed.z, (T)ed.w, pi);
+                st4<T>(tab + r * 4, va);
+            } else if (ty == OP_TS && r < 4) {
+                tipvec<T>(va, r, (T)ed.x, (T)ed.y, pi);
+                st4<T>(tab + r * 4, va);
+            } else if (ty == OP_TTT) {
+                const E4 e1 = s_e[ox.z + 1];
+                tipvec<T>(va, r >> 2, (T)ed.x, (T)ed.y, pi);
+                tipvec<T>(vb, r & 3, (T)ed.z, (T)ed.w, pi);
+#pragma unroll
+                for (int X = 0; X < 4; ++X) va[X] *= vb[X];
+                branch<T>(va, (T)e1.z, (T)e1.w, pi);
+#pragma unroll
+                for (int xc = 0; xc < 4; ++xc) {
+                    tipvec<T>(vb, xc, (T)e1.x, (T)e1.y, pi);
+#pragma unroll
+                    for (int X = 0; X < 4; ++X) vb[X] *= va[X];
+                    st4<T>(tab + (r * 4 + xc) * 4, vb);
+                }
+            }
         }
     }
     __syncthreads();
-    // flag cherry tables with an entry whose max is below the rescale threshold
-    for (int op = tid; op < nops && PT; op += PRUNE_THREADS) {
-        if ((s_op[op].x & 3u) != OP_TT) continue;
-        const T* tab = reinterpret_cast<const T*>(reinterpret_cast<const char*>(s_tab) + s_op[op].y);
+    if constexpr (sparse_checks<T>()) {  // merge the flags (ordered before the op loop by the batch barrier)
+        for (int op = tid; op < nops_c; op += PRUNE_THREADS)
+            if (s_chk[op]) s_opc[op].h.x |= OP_CHECK;
+    }
+    // 4. (every-node checks, FP32) flag the cherry / triplet tables holding a small vector
+    for (int op = tid; op < nops_c && PT && !sparse_checks<T>(); op += PRUNE_THREADS) {
+        const uint32_t ty = s_opc[op].h.x & 3u;
+        if (ty != OP_TT && ty != OP_TTT) continue;
+        const T* tab = reinterpret_cast<const T*>(reinterpret_cast<const char*>(s_tab) + s_opc[op].h.y);
         bool small = false;
-        for (int e = 0; e < 16; ++e) {
+        for (int e = 0; e < (ty == OP_TTT ? 64 : 16); ++e) {
             T v[4];
             ld4<T>(v, tab + 4 * e);
             small |= small4(v);
         }
-        if (small) s_op[op].y |= TAB_CHECK;
+        if (small) s_opc[op].h.y |= TAB_CHECK;
     }
 
     SiteAcc<W> acc;
@@ -651,13 +885,13 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
         int scale[SI];
 #pragma unroll
         for (int k = 0; k < SI; ++k) scale[k] = 0;
-        for (int op = 0; op < nops; ++op) {
-            const uint2 ox = s_op[op];
+        for (int op = 0; op < nops_c; ++op) {
+            const uint4 ox = s_opc[op].h;
             BranchData<T, GM> ed;
-            if constexpr (GM) ed = s_P + op * 32;
-            else ed = s_e[op];
-            const int di = (int)((ox.x >> 2) & 15u) * 3 + (int)(ox.x & 3u);  // dense (sp, type) index
-            run_op<T, DR, SI, PT, DMX, GM>(di, st, ox.x, ox.y, ed, s_tab, cc, pi, scale);
+            if constexpr (GM) ed = s_P + ox.z * 32;
+            else ed = s_opc[op].ed;
+            const int di = (int)((ox.x >> 2) & 15u) * 4 + (int)(ox.x & 3u);  // dense (sp, type) index
+            run_op<T, DR, SI, PT, DMX, GM>(di, st, ox.x, ox.y, ox.w, ed, s_tab, cc, pi, scale);
         }
         const int site0 = s_begin + b * BATCH + tid * SI;
 #pragma unroll
@@ -721,10 +955,48 @@ static cudaError_t launch_flat(const PruneArgs& a, int ntrees, cudaStream_t st) 
                     : launch_flat_w<T, D, false, GM, false>(a, ntrees, st);
 }
 
+// How many triplets the table kernel may fuse: the shared memory left over at the
+// occupancy the kernel reaches without them (registers or base shared memory
+// bound it), so fusion never costs a resident CTA.  Cached per tree size; the
+// first call is at init (mpcgs_init scores G0), outside any graph capture.
+template <typename T, int DR, int SI, bool PT, bool GM, typename K>
+static int tab_trip_cap(K kern, int nops, int need_cap) {
+    if (!PT || MPCGS_NO_TRIPLETS) return 0;
+    static int key[8] = {-1, -1, -1, -1, -1, -1, -1, -1}, val[8];
+    const int k = nops * 16 + need_cap;
+    for (int i = 0; i < 8; ++i)
+        if (key[i] == k) return val[i];
+    const size_t base = tab_smem_bytes<T, DR, SI, PT, GM>(nops, need_cap, 0);
+    int dev = 0, per_sm = 0, resv = 0, optin = 0, blocks = 0;
+    cudaGetDevice(&dev);
+    cudaDeviceGetAttribute(&per_sm, cudaDevAttrMaxSharedMemoryPerMultiprocessor, dev);
+    cudaDeviceGetAttribute(&resv, cudaDevAttrReservedSharedMemoryPerBlock, dev);
+    cudaDeviceGetAttribute(&optin, cudaDevAttrMaxSharedMemoryPerBlockOptin, dev);
+    int cap = 0;
+    cudaFuncAttributes fa{};
+    if (cudaFuncGetAttributes(&fa, kern) == cudaSuccess &&
+        cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, optin - (int)fa.sharedSizeBytes) ==
+            cudaSuccess &&
+        cudaOccupancyMaxActiveBlocksPerMultiprocessor(&blocks, kern, PRUNE_THREADS, base) == cudaSuccess &&
+        blocks > 0) {
+        const long room = std::min<long>(optin, per_sm / blocks - resv - 256) - (long)fa.sharedSizeBytes - (long)base;
+        cap = (int)std::max<long>(0, std::min<long>((nops + 1) / 3, room / (long)(sizeof(T) * TRIP_EXTRA)));
+    }
+    cudaGetLastError();
+    for (int i = 0; i < 8; ++i)
+        if (key[i] < 0) {
+            key[i] = k;
+            val[i] = cap;
+            break;
+        }
+    return cap;
+}
+
 template <typename T, int DR, int SI, bool PT, int DMX, bool W, bool GM>
-static cudaError_t launch_tab_w(const PruneArgs& a, int ntrees, cudaStream_t st) {
-    const size_t smem = tab_smem_bytes<T, DR, SI, PT, GM>(a.nops, a.need_cap);
+static cudaError_t launch_tab_w(PruneArgs a, int ntrees, cudaStream_t st) {
     auto kern = k_prune_tab<T, DR, SI, PT, DMX, W, GM>;
+    a.trip_cap = tab_trip_cap<T, DR, SI, PT, GM>(kern, a.nops, a.need_cap);
+    const size_t smem = tab_smem_bytes<T, DR, SI, PT, GM>(a.nops, a.need_cap, a.trip_cap);
     static size_t attr_bytes = 48 * 1024;
     if (smem > attr_bytes) {
         cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
