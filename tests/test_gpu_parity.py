@@ -177,6 +177,41 @@ def test_underflow_rescaling_long_alignment_many_tips(P, orc):
         assert abs(g - want) <= LL_TOL[prec] * abs(want)
 
 
+@pytest.mark.parametrize("precision", [64, 32])
+@pytest.mark.parametrize("n", [24, 64, 128])
+def test_table_kernel_triplets_and_sparse_checks(P, orc, precision, n):
+    """Table kernel (n <= 128): fused cherry+tip triplet tables and the FP64
+    sparse underflow checks placed by integer bounds (S5).  Trees mix long
+    branches (values fall far below 2^-256 within a subtree, so checks must fire),
+    tiny branches with mismatching tips (the bound's em factor), zero-length
+    branches (no bound: every node checked) and caterpillars (a triplet at the
+    bottom, then a chain of TS ops); L spans several site batches and a ragged tail."""
+    rng = np.random.default_rng(100 + n)
+    L = 1100
+    pi = np.array([0.07, 0.43, 0.38, 0.12])
+    u = orc.default_rate(pi)
+    codes = synth.random_alignment(n, L, rng, pi)
+    trees = [synth.coalescent_tree(n, th, rng) for th in (8.0, 0.3, 1e-4)]
+    for shape in ("caterpillar", "random", "balanced"):
+        p, a = synth.shaped_tree(n, shape, rng, scale=1.0)
+        trees.append((p, a * 3.0))
+    p, a = synth.shaped_tree(n, "random", rng, scale=1.0)
+    a[n:] = np.cumsum(np.where(np.arange(n - 1) % 3 == 0, 1e-7, rng.exponential(2.0, n - 1)))  # tiny and long steps
+    trees.append((p, a))
+    p, a = synth.shaped_tree(n, "caterpillar", rng, scale=1.0)
+    a[n:n + 3] = 0.0  # zero-length branches near the tips
+    trees.append((p, a))
+    ctx = _ctx(P, codes, 0.05, tree=trees[1], precision=precision, base_freq=pi, mu=u, max_proposals=len(trees),
+               max_samples=16)
+    got = ctx.mpcgs_score_trees(np.stack([t[0] for t in trees]), np.stack([t[1] for t in trees]))
+    for k, ((p, a), g) in enumerate(zip(trees, got)):
+        want = orc.log_likelihood(codes, p, a, pi, u)
+        if np.isinf(want):
+            assert g == want, k
+        else:
+            assert abs(g - want) <= LL_TOL[precision] * abs(want), (k, g, want)
+
+
 # ------------------------------------------------------------------ GMH step (lock-step, P20)
 def _lockstep(P, orc, wl, N, steps, seed, K=None, precision=64, incremental=False, compress=False,
               model="F81", kappa=0.0, ambiguity=False):
