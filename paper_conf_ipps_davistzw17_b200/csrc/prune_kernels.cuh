@@ -306,28 +306,58 @@ __device__ __forceinline__ void rescale_sites(T (&v)[SI][4], int (&scale)[SI]) {
     }
 }
 
-// Register stack of DR levels per site, deeper levels in shared memory laid out
-// [level][site k][state X][thread] (conflict-free).
+// Register stack per site.  MPCGS_WINDOW (default): the registers hold the top
+// DR levels (level l in register slot l mod DR, a compile-time index in every
+// (sp, type) case); a push above DR spills the level leaving the window to shared
+// memory and a merge that drops the window below its DR levels fills one back --
+// one vector moved per crossing, not per op.  Otherwise levels >= DR live in shared
+// memory for good.  Shared-memory levels are laid out [level][site k][state X][thread]
+// (conflict-free).
+#ifndef MPCGS_WINDOW
+#define MPCGS_WINDOW 1
+#endif
+
 template <typename T, int DR, int SI>
 struct Stack {
     T r[SI][DR][4];
     T* sm;  // this thread's column of the spill area
+    __device__ __forceinline__ T& smv(int level, int k, int x) const {
+        return sm[((level * SI + k) * 4 + x) * PRUNE_THREADS];
+    }
     template <int S>
     __device__ __forceinline__ void get(int k, T (&v)[4]) const {
-        if constexpr (S < DR) {
-            v[0] = r[k][S][0]; v[1] = r[k][S][1]; v[2] = r[k][S][2]; v[3] = r[k][S][3];
+        if constexpr (MPCGS_WINDOW || S < DR) {
+            constexpr int R = S % DR;
+            v[0] = r[k][R][0]; v[1] = r[k][R][1]; v[2] = r[k][R][2]; v[3] = r[k][R][3];
         } else {
 #pragma unroll
-            for (int x = 0; x < 4; ++x) v[x] = sm[(((S - DR) * SI + k) * 4 + x) * PRUNE_THREADS];
+            for (int x = 0; x < 4; ++x) v[x] = smv(S - DR, k, x);
         }
     }
     template <int S>
     __device__ __forceinline__ void put(int k, const T (&v)[4]) {
-        if constexpr (S < DR) {
-            r[k][S][0] = v[0]; r[k][S][1] = v[1]; r[k][S][2] = v[2]; r[k][S][3] = v[3];
+        if constexpr (MPCGS_WINDOW || S < DR) {
+            constexpr int R = S % DR;
+            r[k][R][0] = v[0]; r[k][R][1] = v[1]; r[k][R][2] = v[2]; r[k][R][3] = v[3];
         } else {
 #pragma unroll
-            for (int x = 0; x < 4; ++x) sm[(((S - DR) * SI + k) * 4 + x) * PRUNE_THREADS] = v[x];
+            for (int x = 0; x < 4; ++x) smv(S - DR, k, x) = v[x];
+        }
+    }
+    // before a push to level S: level S - DR leaves the window (slot S mod DR)
+    template <int S>
+    __device__ __forceinline__ void spill_for_push(int k) {
+        if constexpr (MPCGS_WINDOW && S >= DR) {
+#pragma unroll
+            for (int x = 0; x < 4; ++x) smv(S - DR, k, x) = r[k][S % DR][x];
+        }
+    }
+    // after a merge at stack depth S (levels S-2, S-1 -> S-2): level S-1-DR re-enters
+    template <int S>
+    __device__ __forceinline__ void fill_after_pop(int k) {
+        if constexpr (MPCGS_WINDOW && S - 1 - DR >= 0) {
+#pragma unroll
+            for (int x = 0; x < 4; ++x) r[k][(S - 1) % DR][x] = smv(S - 1 - DR, k, x);
         }
     }
 };
@@ -467,11 +497,10 @@ __device__ void mark_checks(const OpRec<T>* s_opc, const int* s_d, int* s_bnd, u
 
 
 template <typename T, int DR, int SI, bool PT, int S, int DMX>
-__device__ __forceinline__ void tab_tt(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, const T* s_tab,
-                                       const Codes<SI>& c, int (&scale)[SI]) {
+__device__ __forceinline__ void tab_tt(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, uint32_t wa,
+                                       const T* s_tab, const Codes<SI>& c, int (&scale)[SI]) {
     if constexpr (S < DMX) {
         constexpr int EB = 4 * sizeof(T);
-        const uint32_t wa = c.word((code >> 6) & 2047);
         const uint32_t wb = c.word((code >> 17) & 2047);
         const char* base = reinterpret_cast<const char*>(s_tab) + (toff & ~TAB_CHECK);
         T v[SI][4];
@@ -492,17 +521,19 @@ __device__ __forceinline__ void tab_tt(Stack<T, DR, SI>& st, uint32_t code, uint
             if (!sparse_checks<T>() || (code & OP_CHECK)) rescale_sites<T, SI>(v, scale);
         }
 #pragma unroll
-        for (int k = 0; k < SI; ++k) st.template put<S>(k, v[k]);
+        for (int k = 0; k < SI; ++k) {
+            st.template spill_for_push<S>(k);
+            st.template put<S>(k, v[k]);
+        }
     }
 }
 
 // fused triplet: one lookup in the 64x4 table of tip(c) (.) branch(tip(a) (.) tip(b))
 template <typename T, int DR, int SI, bool PT, int S, int DMX>
 __device__ __forceinline__ void tab_ttt(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, uint32_t tc,
-                                        const T* s_tab, const Codes<SI>& c, int (&scale)[SI]) {
+                                        uint32_t wa, const T* s_tab, const Codes<SI>& c, int (&scale)[SI]) {
     if constexpr (PT && S < DMX) {
         constexpr int EB = 4 * sizeof(T);
-        const uint32_t wa = c.word((code >> 6) & 2047);
         const uint32_t wb = c.word((code >> 17) & 2047);
         const uint32_t wc = c.word((int)tc);
         const char* base = reinterpret_cast<const char*>(s_tab) + (toff & ~TAB_CHECK);
@@ -513,7 +544,10 @@ __device__ __forceinline__ void tab_ttt(Stack<T, DR, SI>& st, uint32_t code, uin
                                                     c.template off4<EB>(wb, k) + c.template off<EB>(wc, k)));
         if (sparse_checks<T>() ? (code & OP_CHECK) != 0u : (toff & TAB_CHECK) != 0u) rescale_sites<T, SI>(v, scale);
 #pragma unroll
-        for (int k = 0; k < SI; ++k) st.template put<S>(k, v[k]);
+        for (int k = 0; k < SI; ++k) {
+            st.template spill_for_push<S>(k);
+            st.template put<S>(k, v[k]);
+        }
     }
 }
 
@@ -542,12 +576,12 @@ struct ChildBr {
 };
 
 template <typename T, int DR, int SI, int S, int DMX, bool GM>
-__device__ __forceinline__ void tab_ts(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff,
+__device__ __forceinline__ void tab_ts(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, uint32_t wa,
                                        const BranchData<T, GM>& ed, const T* s_tab, const Codes<SI>& c,
                                        const T (&pi)[4], int (&scale)[SI]) {
     if constexpr (S >= 1 && S <= DMX) {
         constexpr int EB = 4 * sizeof(T);
-        const uint32_t wa = c.word((code >> 6) & 2047);
+        
         const char* base = reinterpret_cast<const char*>(s_tab) + toff;
         const ChildBr<T, GM, true> cb(ed);
         T v[SI][4];
@@ -585,15 +619,18 @@ __device__ __forceinline__ void tab_ss(Stack<T, DR, SI>& st, uint32_t code, cons
         }
         if (!sparse_checks<T>() || (code & OP_CHECK)) rescale_sites<T, SI>(v, scale);
 #pragma unroll
-        for (int k = 0; k < SI; ++k) st.template put<S - 2>(k, v[k]);
+        for (int k = 0; k < SI; ++k) {
+            st.template put<S - 2>(k, v[k]);
+            st.template fill_after_pop<S>(k);
+        }
     }
 }
 
 #define MPCGS_TABCASE(S)                                                                          \
-    case 4 * (S) + 0: tab_tt<T, DR, SI, PT, S, DMX>(st, code, toff, s_tab, cc, scale); break;       \
-    case 4 * (S) + 1: tab_ts<T, DR, SI, S, DMX, GM>(st, code, toff, ed, s_tab, cc, pi, scale); break; \
-    case 4 * (S) + 2: tab_ss<T, DR, SI, S, DMX, GM>(st, code, ed, pi, scale); break;                  \
-    case 4 * (S) + 3: tab_ttt<T, DR, SI, PT, S, DMX>(st, code, toff, tc, s_tab, cc, scale); break;
+    case 4 * (S) + 0: tab_tt<T, DR, SI, PT, S, DMX>(st, code, toff, wa, s_tab, cc, scale); break;       \
+    case 4 * (S) + 1: tab_ts<T, DR, SI, S, DMX, GM>(st, code, toff, wa, ed, s_tab, cc, pi, scale); break; \
+    case 4 * (S) + 2: tab_ss<T, DR, SI, S, DMX, GM>(st, code, ed, pi, scale); break;                      \
+    case 4 * (S) + 3: tab_ttt<T, DR, SI, PT, S, DMX>(st, code, toff, tc, wa, s_tab, cc, scale); break;
 #define MPCGS_CASES_4 MPCGS_TABCASE(0) MPCGS_TABCASE(1) MPCGS_TABCASE(2) MPCGS_TABCASE(3) MPCGS_TABCASE(4)
 #define MPCGS_CASES_6 MPCGS_CASES_4 MPCGS_TABCASE(5) MPCGS_TABCASE(6)
 #define MPCGS_CASES_8 MPCGS_CASES_6 MPCGS_TABCASE(7) MPCGS_TABCASE(8)
@@ -602,7 +639,7 @@ __device__ __forceinline__ void tab_ss(Stack<T, DR, SI>& st, uint32_t code, cons
 // one op for SI sites; the switch only has the (sp, type) labels a DMX-level tree can use
 template <typename T, int DR, int SI, bool PT, int DMX, bool GM>
 __device__ __forceinline__ void run_op(int di, Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, uint32_t tc,
-                                       const BranchData<T, GM>& ed, const T* s_tab, const Codes<SI>& cc,
+                                       uint32_t wa, const BranchData<T, GM>& ed, const T* s_tab, const Codes<SI>& cc,
                                        const T (&pi)[4], int (&scale)[SI]) {
     if constexpr (DMX <= 4) {
         switch (di) { MPCGS_CASES_4 default: __builtin_unreachable(); }
@@ -891,7 +928,8 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
             if constexpr (GM) ed = s_P + ox.z * 32;
             else ed = s_opc[op].ed;
             const int di = (int)((ox.x >> 2) & 15u) * 4 + (int)(ox.x & 3u);  // dense (sp, type) index
-            run_op<T, DR, SI, PT, DMX, GM>(di, st, ox.x, ox.y, ox.w, ed, s_tab, cc, pi, scale);
+            run_op<T, DR, SI, PT, DMX, GM>(di, st, ox.x, ox.y, ox.w, cc.word((ox.x >> 6) & 2047), ed, s_tab, cc, pi,
+                                           scale);
         }
         const int site0 = s_begin + b * BATCH + tid * SI;
 #pragma unroll
