@@ -446,12 +446,12 @@ void upgma(int n, int L, const uint8_t* codes, double theta0, int32_t* parent, d
     }
 }
 
-// Sites per CTA: a multiple of the kernel's site batch (up to 16 batches: amortises the
+// Sites per CTA: a multiple of the kernel's site batch (up to 32 batches: amortises the
 // per-CTA table setup), as many batches as keep
 // >= ~8 CTAs per SM busy.  Depends only on L and the GLOBAL tree count, so every
 // rank tiles (and sums) a proposal's sites identically (world-size invariance).
 #ifndef MPCGS_MAXPER
-#define MPCGS_MAXPER 16
+#define MPCGS_MAXPER 32
 #endif
 void prune_tiling(int n, int L, int ntrees_global, int precision, int& tiles, int& sites_per_cta) {
     const int batch = prune_batch_sites(n, precision);
