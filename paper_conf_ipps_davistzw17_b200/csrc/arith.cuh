@@ -48,18 +48,12 @@ __device__ __forceinline__ void maybe_rescale(float (&v)[4], int& scale) {
 // branch(L)_X = sum_Y P_XY(t) L_Y = e L_X + em (pi . L)   (Eq. 19 + Eq. 20)
 template <typename T>
 __device__ __forceinline__ void branch(T (&r)[4], T e, T em, const T (&pi)[4]) {
-    T t;
-    if constexpr (sizeof(T) == 8) {  // FP64 (latency-bound): pi . L as a depth-3 tree
-        const T s01 = fma(pi[1], r[1], pi[0] * r[0]);
-        const T s23 = fma(pi[3], r[3], pi[2] * r[2]);
-        t = em * (s01 + s23);
-    } else {                         // FP32 (issue-bound): fewest instructions
-        T s = pi[0] * r[0];
-        s = fma(pi[1], r[1], s);
-        s = fma(pi[2], r[2], s);
-        s = fma(pi[3], r[3], s);
-        t = em * s;
-    }
+    // sequential pi . L (fewest FP instructions; four sites per thread supply the ILP)
+    T s = pi[0] * r[0];
+    s = fma(pi[1], r[1], s);
+    s = fma(pi[2], r[2], s);
+    s = fma(pi[3], r[3], s);
+    const T t = em * s;
     r[0] = fma(e, r[0], t);
     r[1] = fma(e, r[1], t);
     r[2] = fma(e, r[2], t);

@@ -994,11 +994,15 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
                 padded[(size_t)i * c->Lpad + site] = (uint8_t)(any_amb ? base_set(cd) : cd);
             }
         const int W2 = codes2_words(L);
+        const int si2 = prune_batch_sites(n, c->precision) / PRUNE_THREADS;  // sites per thread of the table kernel
         std::vector<uint32_t> packed((size_t)n * W2, 0u);
         if (!any_amb)
             for (int i = 0; i < n; ++i)
-                for (int site = 0; site < L; ++site)
-                    packed[(size_t)i * W2 + (site >> 4)] |= (uint32_t)codes[(size_t)i * L + site] << (2 * (site & 15));
+                for (int site = 0; site < L; ++site) {  // thread-interleaved order of the table kernel (Codes)
+                    const int s16 = site & 15, q = s16 / si2, k = s16 % si2;
+                    packed[(size_t)i * W2 + (site >> 4)] |= (uint32_t)codes[(size_t)i * L + site]
+                                                            << ((32 / si2) * k + 2 * q);
+                }
         if (cudaMemcpyAsync((void*)s.codes, padded.data(), padded.size(), cudaMemcpyHostToDevice, c->work) != cudaSuccess ||
             (c->codes2 &&
              cudaMemcpyAsync(c->codes2, packed.data(), packed.size() * 4, cudaMemcpyHostToDevice, c->work) != cudaSuccess)) {

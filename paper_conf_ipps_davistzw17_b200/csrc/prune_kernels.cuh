@@ -362,38 +362,34 @@ struct Stack {
     }
 };
 
-// Tip codes of the current site batch in shared memory, 2-bit packed (16 sites
-// per 32-bit word, a thread's SI sites adjacent).  The byte offset of a site's
-// table entry is one funnel rotation and one mask: rotating the word right by
-// (bit position - log2(entry bytes)) puts the 2-bit code at the entry-size bit.
+// Tip codes of the current site batch in shared memory, 2-bit packed, 16 sites
+// per 32-bit word in the "thread-interleaved" order the host packs (codes2_pack):
+// the word covering threads q = 0..16/SI-1 (SI sites each) holds site k of
+// thread q at bit (32/SI) k + 2 q.  One shift and one mask leave a thread's SI
+// codes as bytes (SI = 4: bytes 0..3; SI = 2: bytes 0 and 2), so the entry index
+// of a cherry (4 a + b) or a fused triplet (16 a + 4 b + c) is formed for all SI
+// sites at once with byte-lane arithmetic (no carries: every lane stays < 64).
 template <int SI>
 struct Codes {
     const unsigned char* base;  // this batch's buffer
     int wofs;                   // word index of this thread's sites
-    uint32_t rb[SI], ra[SI];    // rotations for the code * EB and code * 4 * EB offsets
+    uint32_t qs;                // 2 q: this thread's bit offset in its word
     static constexpr int BATCH = PRUNE_THREADS * SI;
     static constexpr int WB = BATCH / 16;
-    template <int EB>
+    static constexpr uint32_t MASK = SI == 4 ? 0x03030303u : 0x00030003u;
     __device__ __forceinline__ void init(int tid) {
-        constexpr int LG = EB == 32 ? 5 : 4;
         wofs = (tid * SI) >> 4;
-#pragma unroll
-        for (int k = 0; k < SI; ++k) {
-            const int p = ((tid * SI) & 15) * 2 + 2 * k;  // bit position of site k's code
-            rb[k] = (uint32_t)(p - LG) & 31u;
-            ra[k] = (uint32_t)(p - LG - 2) & 31u;
-        }
+        qs = 2u * (uint32_t)(tid % (16 / SI));
     }
     __device__ __forceinline__ uint32_t word(int tip) const {
         return reinterpret_cast<const uint32_t*>(base)[tip * WB + wofs];
     }
+    // this thread's SI codes of a word, one per byte lane
+    __device__ __forceinline__ uint32_t lanes(uint32_t w) const { return (w >> qs) & MASK; }
+    // byte offset of site k's entry in a table of EB-byte entries indexed by the lanes value
     template <int EB>
-    __device__ __forceinline__ uint32_t off(uint32_t w, int k) const {  // code * EB
-        return __funnelshift_r(w, w, rb[k]) & (3u * EB);
-    }
-    template <int EB>
-    __device__ __forceinline__ uint32_t off4(uint32_t w, int k) const {  // code * 4 * EB
-        return __funnelshift_r(w, w, ra[k]) & (12u * EB);
+    __device__ __forceinline__ uint32_t off(uint32_t ln, int k) const {
+        return __byte_perm(ln, 0u, 0x4440u + (uint32_t)(k * (4 / SI))) * (uint32_t)EB;
     }
     static constexpr size_t buf_bytes(int n) { return (size_t)n * WB * 4; }
 };
@@ -504,17 +500,18 @@ __device__ __forceinline__ void tab_tt(Stack<T, DR, SI>& st, uint32_t code, uint
         const uint32_t wb = c.word((code >> 17) & 2047);
         const char* base = reinterpret_cast<const char*>(s_tab) + (toff & ~TAB_CHECK);
         T v[SI][4];
-        if constexpr (PT) {  // 16x4 product table of the cherry
+        if constexpr (PT) {  // 16x4 product table of the cherry, entry 4 x_a + x_b
+            const uint32_t ix = (c.lanes(wa) << 2) + c.lanes(wb);
 #pragma unroll
-            for (int k = 0; k < SI; ++k)
-                ld4<T>(v[k], reinterpret_cast<const T*>(base + c.template off4<EB>(wa, k) + c.template off<EB>(wb, k)));
+            for (int k = 0; k < SI; ++k) ld4<T>(v[k], reinterpret_cast<const T*>(base + c.template off<EB>(ix, k)));
             if (sparse_checks<T>() ? (code & OP_CHECK) != 0u : (toff & TAB_CHECK) != 0u) rescale_sites<T, SI>(v, scale);
         } else {             // two 4x4 tip tables, multiplied here
+            const uint32_t la = c.lanes(wa), lb = c.lanes(wb);
 #pragma unroll
             for (int k = 0; k < SI; ++k) {
                 T w[4];
-                ld4<T>(v[k], reinterpret_cast<const T*>(base + c.template off<EB>(wa, k)));
-                ld4<T>(w, reinterpret_cast<const T*>(base + 16 * sizeof(T) + c.template off<EB>(wb, k)));
+                ld4<T>(v[k], reinterpret_cast<const T*>(base + c.template off<EB>(la, k)));
+                ld4<T>(w, reinterpret_cast<const T*>(base + 16 * sizeof(T) + c.template off<EB>(lb, k)));
 #pragma unroll
                 for (int i = 0; i < 4; ++i) v[k][i] *= w[i];
             }
@@ -538,10 +535,9 @@ __device__ __forceinline__ void tab_ttt(Stack<T, DR, SI>& st, uint32_t code, uin
         const uint32_t wc = c.word((int)tc);
         const char* base = reinterpret_cast<const char*>(s_tab) + (toff & ~TAB_CHECK);
         T v[SI][4];
+        const uint32_t ix = (c.lanes(wa) << 4) + (c.lanes(wb) << 2) + c.lanes(wc);  // entry 16 x_a + 4 x_b + x_c
 #pragma unroll
-        for (int k = 0; k < SI; ++k)
-            ld4<T>(v[k], reinterpret_cast<const T*>(base + (c.template off4<EB>(wa, k) << 2) +
-                                                    c.template off4<EB>(wb, k) + c.template off<EB>(wc, k)));
+        for (int k = 0; k < SI; ++k) ld4<T>(v[k], reinterpret_cast<const T*>(base + c.template off<EB>(ix, k)));
         if (sparse_checks<T>() ? (code & OP_CHECK) != 0u : (toff & TAB_CHECK) != 0u) rescale_sites<T, SI>(v, scale);
 #pragma unroll
         for (int k = 0; k < SI; ++k) {
@@ -583,12 +579,13 @@ __device__ __forceinline__ void tab_ts(Stack<T, DR, SI>& st, uint32_t code, uint
         constexpr int EB = 4 * sizeof(T);
         
         const char* base = reinterpret_cast<const char*>(s_tab) + toff;
+        const uint32_t la = c.lanes(wa);
         const ChildBr<T, GM, true> cb(ed);
         T v[SI][4];
 #pragma unroll
         for (int k = 0; k < SI; ++k) {
             T tip[4];
-            ld4<T>(tip, reinterpret_cast<const T*>(base + c.template off<EB>(wa, k)));
+            ld4<T>(tip, reinterpret_cast<const T*>(base + c.template off<EB>(la, k)));
             st.template get<S - 1>(k, v[k]);
             cb.apply(v[k], pi);
 #pragma unroll
@@ -909,7 +906,7 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
             for (int j = 0; j < 4; ++j) st.r[k][i][j] = T(0);
 
     CD cc;
-    cc.template init<4 * sizeof(T)>(tid);
+    cc.init(tid);
     for (int b = 0; b < nb; ++b) {
         if (b + 1 < nb) {
             issue(b + 1, (b + 1) & 1);

@@ -1,5 +1,5 @@
 #!/bin/bash
-OUT=gpurun_out/sweep_${1:-x}.jsonl; : > $OUT
+OUT=gpurun_out/sweep_inc_${1:-x}.jsonl; : > $OUT
 run() { timeout 300 python bench.py --cpu-seconds 0 --no-e2e --no-incremental-block --steps ${STEPS:-10} --warmup 3 "$@" 2>/dev/null | tail -1 >> $OUT; }
 for inc in "" "--incremental"; do
 run --workload c2 $inc
