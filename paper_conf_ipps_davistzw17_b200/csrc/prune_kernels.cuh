@@ -492,19 +492,50 @@ __device__ void mark_checks(const OpRec<T>* s_opc, const int* s_d, int* s_bnd, u
 }
 
 
-template <typename T, int DR, int SI, bool PT, int S, int DMX>
+// Every op pushes its node's vector already transformed by the node's own
+// parent branch ("up" branch: branch(v)_X = sum_Y P_XY(t_up) v_Y, Eq. 19-20),
+// so each edge of the tree is applied exactly once, by the op below it.  A
+// cherry or fused-triplet table therefore stores branch_up(entry) -- its up
+// branch costs nothing per site -- unless the table holds a vector small
+// enough to need a rescale (TAB_CHECK, rare): then the raw entry is loaded,
+// checked and transformed per site.  The up branch of the root op is the
+// identity (e = 1, em = 0 / P = I), which leaves the root vector unchanged.
+template <typename T, bool GM>
+struct UpBr {
+    std::conditional_t<GM, const T*, T> e;
+    T em;
+    __device__ __forceinline__ UpBr(const typename Traits<T>::E4& ed, const T* s_P) {
+        if constexpr (GM) {
+            e = s_P + (int)ed.x;
+        } else {
+            e = ed.x;
+            em = ed.y;
+        }
+    }
+    __device__ __forceinline__ void apply(T (&v)[4], const T (&pi)[4]) const {
+        if constexpr (GM) gm_branch<T>(v, e);
+        else branch<T>(v, e, em, pi);
+    }
+};
+
+template <typename T, int DR, int SI, bool PT, int S, int DMX, bool GM>
 __device__ __forceinline__ void tab_tt(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, uint32_t wa,
-                                       const T* s_tab, const Codes<SI>& c, int (&scale)[SI]) {
+                                       const UpBr<T, GM>& ub, const T* s_tab, const Codes<SI>& c,
+                                       const T (&pi)[4], int (&scale)[SI]) {
     if constexpr (S < DMX) {
         constexpr int EB = 4 * sizeof(T);
         const uint32_t wb = c.word((code >> 17) & 2047);
         const char* base = reinterpret_cast<const char*>(s_tab) + (toff & ~TAB_CHECK);
         T v[SI][4];
-        if constexpr (PT) {  // 16x4 product table of the cherry, entry 4 x_a + x_b
+        if constexpr (PT) {  // 16x4 table of the cherry, entry 4 x_a + x_b: branch_up(tip_a (.) tip_b)
             const uint32_t ix = (c.lanes(wa) << 2) + c.lanes(wb);
 #pragma unroll
             for (int k = 0; k < SI; ++k) ld4<T>(v[k], reinterpret_cast<const T*>(base + c.template off<EB>(ix, k)));
-            if (sparse_checks<T>() ? (code & OP_CHECK) != 0u : (toff & TAB_CHECK) != 0u) rescale_sites<T, SI>(v, scale);
+            if (toff & TAB_CHECK) {  // raw table: check, then the up branch per site
+                rescale_sites<T, SI>(v, scale);
+#pragma unroll
+                for (int k = 0; k < SI; ++k) ub.apply(v[k], pi);
+            }
         } else {             // two 4x4 tip tables, multiplied here
             const uint32_t la = c.lanes(wa), lb = c.lanes(wb);
 #pragma unroll
@@ -516,6 +547,8 @@ __device__ __forceinline__ void tab_tt(Stack<T, DR, SI>& st, uint32_t code, uint
                 for (int i = 0; i < 4; ++i) v[k][i] *= w[i];
             }
             if (!sparse_checks<T>() || (code & OP_CHECK)) rescale_sites<T, SI>(v, scale);
+#pragma unroll
+            for (int k = 0; k < SI; ++k) ub.apply(v[k], pi);
         }
 #pragma unroll
         for (int k = 0; k < SI; ++k) {
@@ -525,10 +558,11 @@ __device__ __forceinline__ void tab_tt(Stack<T, DR, SI>& st, uint32_t code, uint
     }
 }
 
-// fused triplet: one lookup in the 64x4 table of tip(c) (.) branch(tip(a) (.) tip(b))
-template <typename T, int DR, int SI, bool PT, int S, int DMX>
+// fused triplet: one lookup in the 64x4 table of branch_up(tip(c) (.) branch(tip(a) (.) tip(b)))
+template <typename T, int DR, int SI, bool PT, int S, int DMX, bool GM>
 __device__ __forceinline__ void tab_ttt(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, uint32_t tc,
-                                        uint32_t wa, const T* s_tab, const Codes<SI>& c, int (&scale)[SI]) {
+                                        uint32_t wa, const UpBr<T, GM>& ub, const T* s_tab, const Codes<SI>& c,
+                                        const T (&pi)[4], int (&scale)[SI]) {
     if constexpr (PT && S < DMX) {
         constexpr int EB = 4 * sizeof(T);
         const uint32_t wb = c.word((code >> 17) & 2047);
@@ -538,7 +572,11 @@ __device__ __forceinline__ void tab_ttt(Stack<T, DR, SI>& st, uint32_t code, uin
         const uint32_t ix = (c.lanes(wa) << 4) + (c.lanes(wb) << 2) + c.lanes(wc);  // entry 16 x_a + 4 x_b + x_c
 #pragma unroll
         for (int k = 0; k < SI; ++k) ld4<T>(v[k], reinterpret_cast<const T*>(base + c.template off<EB>(ix, k)));
-        if (sparse_checks<T>() ? (code & OP_CHECK) != 0u : (toff & TAB_CHECK) != 0u) rescale_sites<T, SI>(v, scale);
+        if (toff & TAB_CHECK) {
+            rescale_sites<T, SI>(v, scale);
+#pragma unroll
+            for (int k = 0; k < SI; ++k) ub.apply(v[k], pi);
+        }
 #pragma unroll
         for (int k = 0; k < SI; ++k) {
             st.template spill_for_push<S>(k);
@@ -547,76 +585,51 @@ __device__ __forceinline__ void tab_ttt(Stack<T, DR, SI>& st, uint32_t code, uin
     }
 }
 
-// branch data of an op: F81 {e_a, em_a, e_b, em_b}; general model (f4) a pointer
-// to the op's {P_a, P_b} in shared memory
-template <typename T, bool GM>
-using BranchData = std::conditional_t<GM, const T*, typename Traits<T>::E4>;
-
-// the branch data of one child, loaded once per op (outside the per-site loop)
-template <typename T, bool GM, bool SECOND>
-struct ChildBr {
-    std::conditional_t<GM, const T*, T> e;
-    T em;
-    __device__ __forceinline__ ChildBr(const BranchData<T, GM>& bd) {
-        if constexpr (GM) {
-            e = bd + (SECOND ? 16 : 0);
-        } else {
-            e = SECOND ? bd.z : bd.x;
-            em = SECOND ? bd.w : bd.y;
-        }
-    }
-    __device__ __forceinline__ void apply(T (&v)[4], const T (&pi)[4]) const {
-        if constexpr (GM) gm_branch<T>(v, e);
-        else branch<T>(v, e, em, pi);
-    }
-};
-
+// tip a joined to the stack top (already carrying its branch): v = top (.) tip_a(x_a)
 template <typename T, int DR, int SI, int S, int DMX, bool GM>
 __device__ __forceinline__ void tab_ts(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, uint32_t wa,
-                                       const BranchData<T, GM>& ed, const T* s_tab, const Codes<SI>& c,
+                                       const UpBr<T, GM>& ub, const T* s_tab, const Codes<SI>& c,
                                        const T (&pi)[4], int (&scale)[SI]) {
     if constexpr (S >= 1 && S <= DMX) {
         constexpr int EB = 4 * sizeof(T);
-        
         const char* base = reinterpret_cast<const char*>(s_tab) + toff;
         const uint32_t la = c.lanes(wa);
-        const ChildBr<T, GM, true> cb(ed);
         T v[SI][4];
 #pragma unroll
         for (int k = 0; k < SI; ++k) {
             T tip[4];
             ld4<T>(tip, reinterpret_cast<const T*>(base + c.template off<EB>(la, k)));
             st.template get<S - 1>(k, v[k]);
-            cb.apply(v[k], pi);
 #pragma unroll
             for (int i = 0; i < 4; ++i) v[k][i] *= tip[i];
         }
         if (!sparse_checks<T>() || (code & OP_CHECK)) rescale_sites<T, SI>(v, scale);
 #pragma unroll
-        for (int k = 0; k < SI; ++k) st.template put<S - 1>(k, v[k]);
+        for (int k = 0; k < SI; ++k) {
+            ub.apply(v[k], pi);
+            st.template put<S - 1>(k, v[k]);
+        }
     }
 }
 
+// two stack entries (each already carrying its branch): v = second (.) top
 template <typename T, int DR, int SI, int S, int DMX, bool GM>
-__device__ __forceinline__ void tab_ss(Stack<T, DR, SI>& st, uint32_t code, const BranchData<T, GM>& ed,
+__device__ __forceinline__ void tab_ss(Stack<T, DR, SI>& st, uint32_t code, const UpBr<T, GM>& ub,
                                        const T (&pi)[4], int (&scale)[SI]) {
     if constexpr (S >= 2 && S <= DMX) {
-        const ChildBr<T, GM, false> ca(ed);
-        const ChildBr<T, GM, true> cb(ed);
         T v[SI][4];
 #pragma unroll
         for (int k = 0; k < SI; ++k) {
             T w[4];
             st.template get<S - 2>(k, v[k]);
             st.template get<S - 1>(k, w);
-            ca.apply(v[k], pi);
-            cb.apply(w, pi);
 #pragma unroll
             for (int i = 0; i < 4; ++i) v[k][i] *= w[i];
         }
         if (!sparse_checks<T>() || (code & OP_CHECK)) rescale_sites<T, SI>(v, scale);
 #pragma unroll
         for (int k = 0; k < SI; ++k) {
+            ub.apply(v[k], pi);
             st.template put<S - 2>(k, v[k]);
             st.template fill_after_pop<S>(k);
         }
@@ -624,10 +637,10 @@ __device__ __forceinline__ void tab_ss(Stack<T, DR, SI>& st, uint32_t code, cons
 }
 
 #define MPCGS_TABCASE(S)                                                                          \
-    case 4 * (S) + 0: tab_tt<T, DR, SI, PT, S, DMX>(st, code, toff, wa, s_tab, cc, scale); break;       \
-    case 4 * (S) + 1: tab_ts<T, DR, SI, S, DMX, GM>(st, code, toff, wa, ed, s_tab, cc, pi, scale); break; \
-    case 4 * (S) + 2: tab_ss<T, DR, SI, S, DMX, GM>(st, code, ed, pi, scale); break;                      \
-    case 4 * (S) + 3: tab_ttt<T, DR, SI, PT, S, DMX>(st, code, toff, tc, wa, s_tab, cc, scale); break;
+    case 4 * (S) + 0: tab_tt<T, DR, SI, PT, S, DMX, GM>(st, code, toff, wa, ub, s_tab, cc, pi, scale); break;       \
+    case 4 * (S) + 1: tab_ts<T, DR, SI, S, DMX, GM>(st, code, toff, wa, ub, s_tab, cc, pi, scale); break; \
+    case 4 * (S) + 2: tab_ss<T, DR, SI, S, DMX, GM>(st, code, ub, pi, scale); break;                      \
+    case 4 * (S) + 3: tab_ttt<T, DR, SI, PT, S, DMX, GM>(st, code, toff, tc, wa, ub, s_tab, cc, pi, scale); break;
 #define MPCGS_CASES_4 MPCGS_TABCASE(0) MPCGS_TABCASE(1) MPCGS_TABCASE(2) MPCGS_TABCASE(3) MPCGS_TABCASE(4)
 #define MPCGS_CASES_6 MPCGS_CASES_4 MPCGS_TABCASE(5) MPCGS_TABCASE(6)
 #define MPCGS_CASES_8 MPCGS_CASES_6 MPCGS_TABCASE(7) MPCGS_TABCASE(8)
@@ -636,7 +649,7 @@ __device__ __forceinline__ void tab_ss(Stack<T, DR, SI>& st, uint32_t code, cons
 // one op for SI sites; the switch only has the (sp, type) labels a DMX-level tree can use
 template <typename T, int DR, int SI, bool PT, int DMX, bool GM>
 __device__ __forceinline__ void run_op(int di, Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, uint32_t tc,
-                                       uint32_t wa, const BranchData<T, GM>& ed, const T* s_tab, const Codes<SI>& cc,
+                                       uint32_t wa, const UpBr<T, GM>& ub, const T* s_tab, const Codes<SI>& cc,
                                        const T (&pi)[4], int (&scale)[SI]) {
     if constexpr (DMX <= 4) {
         switch (di) { MPCGS_CASES_4 default: __builtin_unreachable(); }
@@ -657,7 +670,7 @@ template <typename T, int DR, int SI, bool PT, bool GM = false>
 __host__ __device__ size_t tab_smem_bytes(int nops, int need, int trip_cap) {
     const int n = nops + 1;
     const int spill = need > DR ? need - DR : 0;
-    return align16((GM ? 32 * sizeof(T) : sizeof(typename Traits<T>::E4)) * nops) +
+    return align16(GM ? 32 * sizeof(T) * nops + 16 * sizeof(T) : sizeof(typename Traits<T>::E4) * nops) +
            align16(sizeof(T) * ((PT ? 32 : 16) * (size_t)n + (size_t)TRIP_EXTRA * (PT ? trip_cap : 0))) +
            align16(sizeof(OpRec<T>) * nops) + 2 * align16(Codes<SI>::buf_bytes(n)) +
            sizeof(T) * (size_t)spill * SI * 4 * PRUNE_THREADS +
@@ -681,7 +694,8 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
     const int trip_cap = PT ? a.trip_cap : 0;
     E4* s_e = reinterpret_cast<E4*>(smem_raw);  // F81: {e_a, em_a, e_b, em_b} per op
     T* s_P = reinterpret_cast<T*>(smem_raw);    // general model: {P_a, P_b} per op
-    T* s_tab = reinterpret_cast<T*>(smem_raw + align16(OPB * nops));
+    // general model: {P_a, P_b} of every op, then the identity (the root's up branch)
+    T* s_tab = reinterpret_cast<T*>(smem_raw + align16(OPB * nops + (GM ? 16 * sizeof(T) : 0)));
     // compacted ops: {code, table byte offset, original op index, tip c of a fused triplet}
     OpRec<T>* s_opc = reinterpret_cast<OpRec<T>*>(reinterpret_cast<unsigned char*>(s_tab) +
                                             align16(sizeof(T) * (TABE * n + (size_t)TRIP_EXTRA * trip_cap)));
@@ -747,6 +761,7 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
             }
             s_d[i] = Bounds<T>::ilogb(pmin);
         }
+        if (tid < 16) s_P[nops * 32 + tid] = (tid % 5 == 0) ? T(1) : T(0);  // identity: the root's up branch
     }
     __syncthreads();
     // 2. warp 0: fuse the first trip_cap (TT, TS) pairs, compact the op list and
@@ -800,6 +815,38 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
     unsigned char* s_chk = reinterpret_cast<unsigned char*>(s_tl);  // s_code is dead after the scan
     if constexpr (sparse_checks<T>()) {
         if (tid == 32) mark_checks<T>(s_opc, s_d, s_bnd, s_chk, nops_c, Bounds<T>::ilogb(pimin));
+    }
+    //    up branch of every op: the child branch its consumer (the first later op
+    //    that pops the level it pushes) applies to it -- side a of an SS for the
+    //    second entry, side b for the top (SS) or the subtree (TS); none (the
+    //    identity) for the root.  Stored in the op record in place of the
+    //    children's branch data, which the per-site path no longer needs.
+    for (int i = tid; i < nops_c; i += PRUNE_THREADS) {
+        const uint32_t xi = s_opc[i].h.x;
+        const int ty = (int)(xi & 3u), sp = (int)((xi >> 2) & 15u);
+        const int lvl = (ty == (int)OP_TS) ? sp - 1 : (ty == (int)OP_SS ? sp - 2 : sp);
+        E4 up;
+        up.x = GM ? (T)(nops * 32) : T(1);
+        up.y = T(0);
+        up.z = T(0);
+        up.w = T(0);
+        for (int j = i + 1; j < nops_c; ++j) {
+            const uint4 oj = s_opc[j].h;
+            const int tj = (int)(oj.x & 3u), sj = (int)((oj.x >> 2) & 15u);
+            const int side = (tj == (int)OP_TS && sj - 1 == lvl) ? 1
+                             : (tj == (int)OP_SS && sj - 2 == lvl) ? 0
+                             : (tj == (int)OP_SS && sj - 1 == lvl) ? 1 : -1;
+            if (side < 0) continue;
+            if constexpr (GM) {
+                up.x = (T)(oj.z * 32u + (uint32_t)side * 16u);
+            } else {
+                const E4 e = s_e[oj.z];
+                up.x = side ? e.z : e.x;
+                up.y = side ? e.w : e.y;
+            }
+            break;
+        }
+        s_opc[i].ed = up;
     }
     //    tables, one 4-vector (row) per work item: tip tables P_{.,x}(t) (Eq. 19-20 at an
     //    indicator tip), cherry rows tip_a(xa) (.) tip_b(xb), and fused-triplet rows
@@ -881,18 +928,43 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
         for (int op = tid; op < nops_c; op += PRUNE_THREADS)
             if (s_chk[op]) s_opc[op].h.x |= OP_CHECK;
     }
-    // 4. (every-node checks, FP32) flag the cherry / triplet tables holding a small vector
-    for (int op = tid; op < nops_c && PT && !sparse_checks<T>(); op += PRUNE_THREADS) {
-        const uint32_t ty = s_opc[op].h.x & 3u;
-        if (ty != OP_TT && ty != OP_TTT) continue;
-        const T* tab = reinterpret_cast<const T*>(reinterpret_cast<const char*>(s_tab) + s_opc[op].h.y);
-        bool small = false;
-        for (int e = 0; e < (ty == OP_TTT ? 64 : 16); ++e) {
-            T v[4];
-            ld4<T>(v, tab + 4 * e);
-            small |= small4(v);
+    // 4. cherry / triplet tables: fold each op's up branch into its table, unless
+    //    an entry is small enough to need a rescale (max < 2^-TS): that table
+    //    stays raw and is checked and transformed per site (TAB_CHECK).  A half
+    //    warp (16 lanes, rows r) covers one op, so the flag is one ballot.
+    const int nrow = ((nops_c * 16 + 31) / 32) * 32;
+    for (int idx = tid; idx < nrow && PT; idx += PRUNE_THREADS) {
+        const int op = idx >> 4, r = idx & 15;
+        bool tabop = false, small = false;
+        T* tab = nullptr;
+        int ne = 1;
+        if (op < nops_c) {
+            const uint4 ox = s_opc[op].h;
+            const uint32_t ty = ox.x & 3u;
+            tabop = ty == OP_TT || ty == OP_TTT;
+            ne = ty == OP_TTT ? 4 : 1;
+            tab = reinterpret_cast<T*>(reinterpret_cast<char*>(s_tab) + (ox.y & ~TAB_CHECK)) + r * ne * 4;
+            for (int e = 0; e < ne && tabop; ++e) {
+                T v[4];
+                ld4<T>(v, tab + 4 * e);
+                small |= small4(v);
+            }
         }
-        if (small) s_opc[op].h.y |= TAB_CHECK;
+        const unsigned m = __ballot_sync(0xffffffffu, small);
+        const bool raw = ((m >> (tid & 16)) & 0xffffu) != 0u;
+        if (tabop) {
+            if (raw) {
+                if (r == 0) s_opc[op].h.y |= TAB_CHECK;
+            } else {
+                const UpBr<T, GM> ub(s_opc[op].ed, s_P);
+                for (int e = 0; e < ne; ++e) {
+                    T v[4];
+                    ld4<T>(v, tab + 4 * e);
+                    ub.apply(v, pi);
+                    st4<T>(tab + 4 * e, v);
+                }
+            }
+        }
     }
 
     SiteAcc<W> acc;
@@ -921,11 +993,9 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
         for (int k = 0; k < SI; ++k) scale[k] = 0;
         for (int op = 0; op < nops_c; ++op) {
             const uint4 ox = s_opc[op].h;
-            BranchData<T, GM> ed;
-            if constexpr (GM) ed = s_P + ox.z * 32;
-            else ed = s_opc[op].ed;
+            const UpBr<T, GM> ub(s_opc[op].ed, s_P);
             const int di = (int)((ox.x >> 2) & 15u) * 4 + (int)(ox.x & 3u);  // dense (sp, type) index
-            run_op<T, DR, SI, PT, DMX, GM>(di, st, ox.x, ox.y, ox.w, cc.word((ox.x >> 6) & 2047), ed, s_tab, cc, pi,
+            run_op<T, DR, SI, PT, DMX, GM>(di, st, ox.x, ox.y, ox.w, cc.word((ox.x >> 6) & 2047), ub, s_tab, cc, pi,
                                            scale);
         }
         const int site0 = s_begin + b * BATCH + tid * SI;
