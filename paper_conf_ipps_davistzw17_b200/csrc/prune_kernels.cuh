@@ -413,6 +413,11 @@ constexpr uint32_t TAB_CHECK = 0x80000000u;  // toff flag: the cherry table can 
 #define MPCGS_NO_TRIPLETS 0
 #endif
 constexpr uint32_t OP_CHECK = 1u << 28;  // op code flag (bits 28-31 are free): check this op's result
+// op code bits 29-30 of a TS-type op: 0 = tip table, 1 = fused cherry + SS, 2 = fused triplet + SS
+constexpr int OP_FUSED_SHIFT = 29;
+#ifndef MPCGS_FUSE_SS
+#define MPCGS_FUSE_SS 1
+#endif
 // Fused triplet (table kernel only): a cherry (TT, tips a and b) immediately
 // followed by the TS op that joins it to tip c -- one 64x4 table of the result
 // over (x_a, x_b, x_c), built per CTA.  Type 3 is unused by the schedule encoding.
@@ -447,12 +452,12 @@ struct Bounds<float> {
 // compacted op list s_opc (a fused triplet, type OP_TTT, covers original ops o
 // and o+1) and sets s_chk[i] for the ops to check (merged into OP_CHECK later).
 // compacted op record of the table kernel: {code, table byte offset, original op
-// index, tip c of a fused triplet} and the op's F81 branch data (one address, so
-// the two loads of an op do not depend on each other)
+// index, tip c of a fused triplet} and the op's up branch (one address, so the
+// two loads of an op do not depend on each other)
 template <typename T>
 struct __align__(16) OpRec {
     uint4 h;
-    typename Traits<T>::E4 ed;
+    T up[2];  // the op's up branch: F81 {e, em}; general model {offset of P_up in s_P, 0}
 };
 
 template <typename T>
@@ -504,12 +509,12 @@ template <typename T, bool GM>
 struct UpBr {
     std::conditional_t<GM, const T*, T> e;
     T em;
-    __device__ __forceinline__ UpBr(const typename Traits<T>::E4& ed, const T* s_P) {
+    __device__ __forceinline__ UpBr(const T (&up)[2], const T* s_P) {
         if constexpr (GM) {
-            e = s_P + (int)ed.x;
+            e = s_P + (int)up[0];
         } else {
-            e = ed.x;
-            em = ed.y;
+            e = up[0];
+            em = up[1];
         }
     }
     __device__ __forceinline__ void apply(T (&v)[4], const T (&pi)[4]) const {
@@ -585,15 +590,23 @@ __device__ __forceinline__ void tab_ttt(Stack<T, DR, SI>& st, uint32_t code, uin
     }
 }
 
-// tip a joined to the stack top (already carrying its branch): v = top (.) tip_a(x_a)
+// tip a joined to the stack top (already carrying its branch): v = top (.) tip_a(x_a).
+// Fused (OP_FUSED kind 1 / 2): a cherry / triplet table op and the SS that merges
+// its result into the stack top, v = top (.) table(x_a, x_b[, x_c]) -- the table
+// already carries the cherry's branch into the SS, the op record the SS's up branch.
 template <typename T, int DR, int SI, int S, int DMX, bool GM>
-__device__ __forceinline__ void tab_ts(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, uint32_t wa,
-                                       const UpBr<T, GM>& ub, const T* s_tab, const Codes<SI>& c,
+__device__ __forceinline__ void tab_ts(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, uint32_t tc,
+                                       uint32_t wa, const UpBr<T, GM>& ub, const T* s_tab, const Codes<SI>& c,
                                        const T (&pi)[4], int (&scale)[SI]) {
     if constexpr (S >= 1 && S <= DMX) {
         constexpr int EB = 4 * sizeof(T);
-        const char* base = reinterpret_cast<const char*>(s_tab) + toff;
-        const uint32_t la = c.lanes(wa);
+        const char* base = reinterpret_cast<const char*>(s_tab) + (toff & ~TAB_CHECK);
+        uint32_t la = c.lanes(wa);
+        const uint32_t kind = (code >> OP_FUSED_SHIFT) & 3u;
+        if (kind != 0u) {
+            la = (la << 2) + c.lanes(c.word((code >> 17) & 2047));
+            if (kind == 2u) la = (la << 2) + c.lanes(c.word((int)tc));
+        }
         T v[SI][4];
 #pragma unroll
         for (int k = 0; k < SI; ++k) {
@@ -638,7 +651,7 @@ __device__ __forceinline__ void tab_ss(Stack<T, DR, SI>& st, uint32_t code, cons
 
 #define MPCGS_TABCASE(S)                                                                          \
     case 4 * (S) + 0: tab_tt<T, DR, SI, PT, S, DMX, GM>(st, code, toff, wa, ub, s_tab, cc, pi, scale); break;       \
-    case 4 * (S) + 1: tab_ts<T, DR, SI, S, DMX, GM>(st, code, toff, wa, ub, s_tab, cc, pi, scale); break; \
+    case 4 * (S) + 1: tab_ts<T, DR, SI, S, DMX, GM>(st, code, toff, tc, wa, ub, s_tab, cc, pi, scale); break; \
     case 4 * (S) + 2: tab_ss<T, DR, SI, S, DMX, GM>(st, code, ub, pi, scale); break;                      \
     case 4 * (S) + 3: tab_ttt<T, DR, SI, PT, S, DMX, GM>(st, code, toff, tc, wa, ub, s_tab, cc, pi, scale); break;
 #define MPCGS_CASES_4 MPCGS_TABCASE(0) MPCGS_TABCASE(1) MPCGS_TABCASE(2) MPCGS_TABCASE(3) MPCGS_TABCASE(4)
@@ -800,7 +813,6 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
             if (keep) {
                 const uint32_t cx = start ? ((code & ~3u) | OP_TTT) : code;
                 s_opc[j].h = make_uint4(cx, (c_size + x - sz) * (uint32_t)sizeof(T), (uint32_t)i, start ? tc : 0u);
-                if constexpr (!GM) s_opc[j].ed = s_e[i];
             }
             c_size += __shfl_sync(0xffffffffu, x, 31);
             c_keep += __popc(mk);
@@ -825,11 +837,7 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
         const uint32_t xi = s_opc[i].h.x;
         const int ty = (int)(xi & 3u), sp = (int)((xi >> 2) & 15u);
         const int lvl = (ty == (int)OP_TS) ? sp - 1 : (ty == (int)OP_SS ? sp - 2 : sp);
-        E4 up;
-        up.x = GM ? (T)(nops * 32) : T(1);
-        up.y = T(0);
-        up.z = T(0);
-        up.w = T(0);
+        T up0 = GM ? (T)(nops * 32) : T(1), up1 = T(0);
         for (int j = i + 1; j < nops_c; ++j) {
             const uint4 oj = s_opc[j].h;
             const int tj = (int)(oj.x & 3u), sj = (int)((oj.x >> 2) & 15u);
@@ -838,15 +846,16 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
                              : (tj == (int)OP_SS && sj - 1 == lvl) ? 1 : -1;
             if (side < 0) continue;
             if constexpr (GM) {
-                up.x = (T)(oj.z * 32u + (uint32_t)side * 16u);
+                up0 = (T)(oj.z * 32u + (uint32_t)side * 16u);
             } else {
                 const E4 e = s_e[oj.z];
-                up.x = side ? e.z : e.x;
-                up.y = side ? e.w : e.y;
+                up0 = side ? (T)e.z : (T)e.x;
+                up1 = side ? (T)e.w : (T)e.y;
             }
             break;
         }
-        s_opc[i].ed = up;
+        s_opc[i].up[0] = up0;
+        s_opc[i].up[1] = up1;
     }
     //    tables, one 4-vector (row) per work item: tip tables P_{.,x}(t) (Eq. 19-20 at an
     //    indicator tip), cherry rows tip_a(xa) (.) tip_b(xb), and fused-triplet rows
@@ -956,7 +965,7 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
             if (raw) {
                 if (r == 0) s_opc[op].h.y |= TAB_CHECK;
             } else {
-                const UpBr<T, GM> ub(s_opc[op].ed, s_P);
+                const UpBr<T, GM> ub(s_opc[op].up, s_P);
                 for (int e = 0; e < ne; ++e) {
                     T v[4];
                     ld4<T>(v, tab + 4 * e);
@@ -965,6 +974,33 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
                 }
             }
         }
+    }
+    // 5. fuse each folded cherry / triplet op with an SS that immediately merges its
+    //    result: one TS-type op at the table op's depth (top (.) table entry) with the
+    //    SS's check flag and up branch -- one dispatch, push and pop fewer per pair.
+    int nops_run = nops_c;
+    if constexpr (PT && MPCGS_FUSE_SS) {
+        __syncthreads();
+        if (tid == 0) {
+            int j = 0;
+            for (int i = 0; i < nops_c; ++i) {
+                OpRec<T> o = s_opc[i];
+                const uint32_t ty = o.h.x & 3u;
+                if ((ty == OP_TT || ty == OP_TTT) && !(o.h.y & TAB_CHECK) && i + 1 < nops_c &&
+                    (s_opc[i + 1].h.x & 3u) == OP_SS) {
+                    const OpRec<T> ss = s_opc[i + 1];
+                    o.h.x = (o.h.x & ~(3u | OP_CHECK | (3u << OP_FUSED_SHIFT))) | OP_TS | (ss.h.x & OP_CHECK) |
+                            ((ty == OP_TTT ? 2u : 1u) << OP_FUSED_SHIFT);
+                    o.up[0] = ss.up[0];
+                    o.up[1] = ss.up[1];
+                    ++i;
+                }
+                s_opc[j++] = o;
+            }
+            s_nc = j;
+        }
+        __syncthreads();
+        nops_run = s_nc;
     }
 
     SiteAcc<W> acc;
@@ -991,9 +1027,9 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
         int scale[SI];
 #pragma unroll
         for (int k = 0; k < SI; ++k) scale[k] = 0;
-        for (int op = 0; op < nops_c; ++op) {
+        for (int op = 0; op < nops_run; ++op) {
             const uint4 ox = s_opc[op].h;
-            const UpBr<T, GM> ub(s_opc[op].ed, s_P);
+            const UpBr<T, GM> ub(s_opc[op].up, s_P);
             const int di = (int)((ox.x >> 2) & 15u) * 4 + (int)(ox.x & 3u);  // dense (sp, type) index
             run_op<T, DR, SI, PT, DMX, GM>(di, st, ox.x, ox.y, ox.w, cc.word((ox.x >> 6) & 2047), ub, s_tab, cc, pi,
                                            scale);
