@@ -290,6 +290,46 @@ __device__ __forceinline__ void cp_async_commit() { asm volatile("cp.async.commi
 template <int N>
 __device__ __forceinline__ void cp_async_wait() { asm volatile("cp.async.wait_group %0;\n" ::"n"(N)); }
 
+// Shared-memory loads from 32-bit shared-window addresses: the op loop addresses
+// its tables, code words and op records from one base computed before the loop
+// (generic pointers made the compiler re-derive the shared window base per op).
+__device__ __forceinline__ uint32_t smem_addr(const void* p) { return (uint32_t)__cvta_generic_to_shared(p); }
+__device__ __forceinline__ uint32_t lds_u32(uint32_t a) {
+    uint32_t v;
+    asm volatile("ld.shared.u32 %0, [%1];\n" : "=r"(v) : "r"(a));
+    return v;
+}
+__device__ __forceinline__ uint4 lds_u4(uint32_t a) {
+    uint4 v;
+    asm volatile("ld.shared.v4.u32 {%0, %1, %2, %3}, [%4];\n" : "=r"(v.x), "=r"(v.y), "=r"(v.z), "=r"(v.w) : "r"(a));
+    return v;
+}
+__device__ __forceinline__ void lds2(double (&r)[2], uint32_t a) {
+    asm volatile("ld.shared.v2.f64 {%0, %1}, [%2];\n" : "=d"(r[0]), "=d"(r[1]) : "r"(a));
+}
+__device__ __forceinline__ void lds2(float (&r)[2], uint32_t a) {
+    asm volatile("ld.shared.v2.f32 {%0, %1}, [%2];\n" : "=f"(r[0]), "=f"(r[1]) : "r"(a));
+}
+__device__ __forceinline__ double lds1(uint32_t a, double) {
+    double v;
+    asm volatile("ld.shared.f64 %0, [%1];\n" : "=d"(v) : "r"(a));
+    return v;
+}
+__device__ __forceinline__ float lds1(uint32_t a, float) {
+    float v;
+    asm volatile("ld.shared.f32 %0, [%1];\n" : "=f"(v) : "r"(a));
+    return v;
+}
+__device__ __forceinline__ void sts1(uint32_t a, double v) { asm volatile("st.shared.f64 [%0], %1;\n" ::"r"(a), "d"(v)); }
+__device__ __forceinline__ void sts1(uint32_t a, float v) { asm volatile("st.shared.f32 [%0], %1;\n" ::"r"(a), "f"(v)); }
+__device__ __forceinline__ void lds4(double (&r)[4], uint32_t a) {
+    asm volatile("ld.shared.v2.f64 {%0, %1}, [%2];\n" : "=d"(r[0]), "=d"(r[1]) : "r"(a));
+    asm volatile("ld.shared.v2.f64 {%0, %1}, [%2+16];\n" : "=d"(r[2]), "=d"(r[3]) : "r"(a));
+}
+__device__ __forceinline__ void lds4(float (&r)[4], uint32_t a) {
+    asm volatile("ld.shared.v4.f32 {%0, %1, %2, %3}, [%4];\n" : "=f"(r[0]), "=f"(r[1]), "=f"(r[2]), "=f"(r[3]) : "r"(a));
+}
+
 template <typename T, int SI>
 __device__ __forceinline__ void rescale_sites(T (&v)[SI][4], int (&scale)[SI]) {
     bool any = false;
@@ -320,9 +360,9 @@ __device__ __forceinline__ void rescale_sites(T (&v)[SI][4], int (&scale)[SI]) {
 template <typename T, int DR, int SI>
 struct Stack {
     T r[SI][DR][4];
-    T* sm;  // this thread's column of the spill area
-    __device__ __forceinline__ T& smv(int level, int k, int x) const {
-        return sm[((level * SI + k) * 4 + x) * PRUNE_THREADS];
+    uint32_t sm;  // this thread's column of the spill area (shared-window address)
+    __device__ __forceinline__ uint32_t sma(int level, int k, int x) const {
+        return sm + (uint32_t)(((level * SI + k) * 4 + x) * PRUNE_THREADS) * (uint32_t)sizeof(T);
     }
     template <int S>
     __device__ __forceinline__ void get(int k, T (&v)[4]) const {
@@ -331,7 +371,7 @@ struct Stack {
             v[0] = r[k][R][0]; v[1] = r[k][R][1]; v[2] = r[k][R][2]; v[3] = r[k][R][3];
         } else {
 #pragma unroll
-            for (int x = 0; x < 4; ++x) v[x] = smv(S - DR, k, x);
+            for (int x = 0; x < 4; ++x) v[x] = lds1(sma(S - DR, k, x), T(0));
         }
     }
     template <int S>
@@ -341,7 +381,7 @@ struct Stack {
             r[k][R][0] = v[0]; r[k][R][1] = v[1]; r[k][R][2] = v[2]; r[k][R][3] = v[3];
         } else {
 #pragma unroll
-            for (int x = 0; x < 4; ++x) smv(S - DR, k, x) = v[x];
+            for (int x = 0; x < 4; ++x) sts1(sma(S - DR, k, x), v[x]);
         }
     }
     // before a push to level S: level S - DR leaves the window (slot S mod DR)
@@ -349,7 +389,7 @@ struct Stack {
     __device__ __forceinline__ void spill_for_push(int k) {
         if constexpr (MPCGS_WINDOW && S >= DR) {
 #pragma unroll
-            for (int x = 0; x < 4; ++x) smv(S - DR, k, x) = r[k][S % DR][x];
+            for (int x = 0; x < 4; ++x) sts1(sma(S - DR, k, x), r[k][S % DR][x]);
         }
     }
     // after a merge at stack depth S (levels S-2, S-1 -> S-2): level S-1-DR re-enters
@@ -357,7 +397,7 @@ struct Stack {
     __device__ __forceinline__ void fill_after_pop(int k) {
         if constexpr (MPCGS_WINDOW && S - 1 - DR >= 0) {
 #pragma unroll
-            for (int x = 0; x < 4; ++x) r[k][(S - 1) % DR][x] = smv(S - 1 - DR, k, x);
+            for (int x = 0; x < 4; ++x) r[k][(S - 1) % DR][x] = lds1(sma(S - 1 - DR, k, x), T(0));
         }
     }
 };
@@ -371,7 +411,7 @@ struct Stack {
 // sites at once with byte-lane arithmetic (no carries: every lane stays < 64).
 template <int SI>
 struct Codes {
-    const unsigned char* base;  // this batch's buffer
+    uint32_t sbase;             // this batch's buffer (shared-window address)
     int wofs;                   // word index of this thread's sites
     uint32_t qs;                // 2 q: this thread's bit offset in its word
     static constexpr int BATCH = PRUNE_THREADS * SI;
@@ -382,7 +422,7 @@ struct Codes {
         qs = 2u * (uint32_t)(tid % (16 / SI));
     }
     __device__ __forceinline__ uint32_t word(int tip) const {
-        return reinterpret_cast<const uint32_t*>(base)[tip * WB + wofs];
+        return lds_u32(sbase + (uint32_t)(tip * WB + wofs) * 4u);
     }
     // this thread's SI codes of a word, one per byte lane
     __device__ __forceinline__ uint32_t lanes(uint32_t w) const { return (w >> qs) & MASK; }
@@ -525,17 +565,17 @@ struct UpBr {
 
 template <typename T, int DR, int SI, bool PT, int S, int DMX, bool GM>
 __device__ __forceinline__ void tab_tt(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, uint32_t wa,
-                                       const UpBr<T, GM>& ub, const T* s_tab, const Codes<SI>& c,
+                                       const UpBr<T, GM>& ub, uint32_t s_tab, const Codes<SI>& c,
                                        const T (&pi)[4], int (&scale)[SI]) {
     if constexpr (S < DMX) {
         constexpr int EB = 4 * sizeof(T);
         const uint32_t wb = c.word((code >> 17) & 2047);
-        const char* base = reinterpret_cast<const char*>(s_tab) + (toff & ~TAB_CHECK);
+        const uint32_t base = s_tab + (toff & ~TAB_CHECK);
         T v[SI][4];
         if constexpr (PT) {  // 16x4 table of the cherry, entry 4 x_a + x_b: branch_up(tip_a (.) tip_b)
             const uint32_t ix = (c.lanes(wa) << 2) + c.lanes(wb);
 #pragma unroll
-            for (int k = 0; k < SI; ++k) ld4<T>(v[k], reinterpret_cast<const T*>(base + c.template off<EB>(ix, k)));
+            for (int k = 0; k < SI; ++k) lds4(v[k], base + c.template off<EB>(ix, k));
             if (toff & TAB_CHECK) {  // raw table: check, then the up branch per site
                 rescale_sites<T, SI>(v, scale);
 #pragma unroll
@@ -546,8 +586,8 @@ __device__ __forceinline__ void tab_tt(Stack<T, DR, SI>& st, uint32_t code, uint
 #pragma unroll
             for (int k = 0; k < SI; ++k) {
                 T w[4];
-                ld4<T>(v[k], reinterpret_cast<const T*>(base + c.template off<EB>(la, k)));
-                ld4<T>(w, reinterpret_cast<const T*>(base + 16 * sizeof(T) + c.template off<EB>(lb, k)));
+                lds4(v[k], base + c.template off<EB>(la, k));
+                lds4(w, base + 16 * (uint32_t)sizeof(T) + c.template off<EB>(lb, k));
 #pragma unroll
                 for (int i = 0; i < 4; ++i) v[k][i] *= w[i];
             }
@@ -566,17 +606,17 @@ __device__ __forceinline__ void tab_tt(Stack<T, DR, SI>& st, uint32_t code, uint
 // fused triplet: one lookup in the 64x4 table of branch_up(tip(c) (.) branch(tip(a) (.) tip(b)))
 template <typename T, int DR, int SI, bool PT, int S, int DMX, bool GM>
 __device__ __forceinline__ void tab_ttt(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, uint32_t tc,
-                                        uint32_t wa, const UpBr<T, GM>& ub, const T* s_tab, const Codes<SI>& c,
+                                        uint32_t wa, const UpBr<T, GM>& ub, uint32_t s_tab, const Codes<SI>& c,
                                         const T (&pi)[4], int (&scale)[SI]) {
     if constexpr (PT && S < DMX) {
         constexpr int EB = 4 * sizeof(T);
         const uint32_t wb = c.word((code >> 17) & 2047);
         const uint32_t wc = c.word((int)tc);
-        const char* base = reinterpret_cast<const char*>(s_tab) + (toff & ~TAB_CHECK);
+        const uint32_t base = s_tab + (toff & ~TAB_CHECK);
         T v[SI][4];
         const uint32_t ix = (c.lanes(wa) << 4) + (c.lanes(wb) << 2) + c.lanes(wc);  // entry 16 x_a + 4 x_b + x_c
 #pragma unroll
-        for (int k = 0; k < SI; ++k) ld4<T>(v[k], reinterpret_cast<const T*>(base + c.template off<EB>(ix, k)));
+        for (int k = 0; k < SI; ++k) lds4(v[k], base + c.template off<EB>(ix, k));
         if (toff & TAB_CHECK) {
             rescale_sites<T, SI>(v, scale);
 #pragma unroll
@@ -596,11 +636,11 @@ __device__ __forceinline__ void tab_ttt(Stack<T, DR, SI>& st, uint32_t code, uin
 // already carries the cherry's branch into the SS, the op record the SS's up branch.
 template <typename T, int DR, int SI, int S, int DMX, bool GM>
 __device__ __forceinline__ void tab_ts(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, uint32_t tc,
-                                       uint32_t wa, const UpBr<T, GM>& ub, const T* s_tab, const Codes<SI>& c,
+                                       uint32_t wa, const UpBr<T, GM>& ub, uint32_t s_tab, const Codes<SI>& c,
                                        const T (&pi)[4], int (&scale)[SI]) {
     if constexpr (S >= 1 && S <= DMX) {
         constexpr int EB = 4 * sizeof(T);
-        const char* base = reinterpret_cast<const char*>(s_tab) + (toff & ~TAB_CHECK);
+        const uint32_t base = s_tab + (toff & ~TAB_CHECK);
         uint32_t la = c.lanes(wa);
         const uint32_t kind = (code >> OP_FUSED_SHIFT) & 3u;
         if (kind != 0u) {
@@ -611,7 +651,7 @@ __device__ __forceinline__ void tab_ts(Stack<T, DR, SI>& st, uint32_t code, uint
 #pragma unroll
         for (int k = 0; k < SI; ++k) {
             T tip[4];
-            ld4<T>(tip, reinterpret_cast<const T*>(base + c.template off<EB>(la, k)));
+            lds4(tip, base + c.template off<EB>(la, k));
             st.template get<S - 1>(k, v[k]);
 #pragma unroll
             for (int i = 0; i < 4; ++i) v[k][i] *= tip[i];
@@ -662,7 +702,7 @@ __device__ __forceinline__ void tab_ss(Stack<T, DR, SI>& st, uint32_t code, cons
 // one op for SI sites; the switch only has the (sp, type) labels a DMX-level tree can use
 template <typename T, int DR, int SI, bool PT, int DMX, bool GM>
 __device__ __forceinline__ void run_op(int di, Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, uint32_t tc,
-                                       uint32_t wa, const UpBr<T, GM>& ub, const T* s_tab, const Codes<SI>& cc,
+                                       uint32_t wa, const UpBr<T, GM>& ub, uint32_t s_tab, const Codes<SI>& cc,
                                        const T (&pi)[4], int (&scale)[SI]) {
     if constexpr (DMX <= 4) {
         switch (di) { MPCGS_CASES_4 default: __builtin_unreachable(); }
@@ -1005,7 +1045,7 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
 
     SiteAcc<W> acc;
     Stack<T, DR, SI> st;
-    st.sm = s_spill + tid;
+    st.sm = smem_addr(s_spill + tid);
 #pragma unroll
     for (int k = 0; k < SI; ++k)
 #pragma unroll
@@ -1015,6 +1055,7 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
 
     CD cc;
     cc.init(tid);
+    const uint32_t s_tab_a = smem_addr(s_tab), s_opc_a = smem_addr(s_opc);
     for (int b = 0; b < nb; ++b) {
         if (b + 1 < nb) {
             issue(b + 1, (b + 1) & 1);
@@ -1023,16 +1064,19 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
             cp_async_wait<0>();
         }
         __syncthreads();
-        cc.base = s_cod + (size_t)(b & 1) * bufb;
+        cc.sbase = smem_addr(s_cod + (size_t)(b & 1) * bufb);
         int scale[SI];
 #pragma unroll
         for (int k = 0; k < SI; ++k) scale[k] = 0;
         for (int op = 0; op < nops_run; ++op) {
-            const uint4 ox = s_opc[op].h;
-            const UpBr<T, GM> ub(s_opc[op].up, s_P);
+            const uint32_t oa = s_opc_a + (uint32_t)op * (uint32_t)sizeof(OpRec<T>);
+            const uint4 ox = lds_u4(oa);
+            T up[2];
+            lds2(up, oa + 16u);
+            const UpBr<T, GM> ub(up, s_P);
             const int di = (int)((ox.x >> 2) & 15u) * 4 + (int)(ox.x & 3u);  // dense (sp, type) index
-            run_op<T, DR, SI, PT, DMX, GM>(di, st, ox.x, ox.y, ox.w, cc.word((ox.x >> 6) & 2047), ub, s_tab, cc, pi,
-                                           scale);
+            run_op<T, DR, SI, PT, DMX, GM>(di, st, ox.x, ox.y, ox.w, cc.word((ox.x >> 6) & 2047), ub, s_tab_a, cc,
+                                           pi, scale);
         }
         const int site0 = s_begin + b * BATCH + tid * SI;
 #pragma unroll
