@@ -446,14 +446,46 @@ void upgma(int n, int L, const uint8_t* codes, double theta0, int32_t* parent, d
     }
 }
 
-// Sites per CTA: a multiple of the kernel's site batch (up to 32 batches: amortises the
-// per-CTA table setup), as many batches as keep
-// >= ~8 CTAs per SM busy.  Depends only on L and the GLOBAL tree count, so every
-// rank tiles (and sums) a proposal's sites identically (world-size invariance).
+// Sites per CTA: a multiple of the kernel's site batch (1..MPCGS_MAXPER batches),
+// chosen by a small cost model in units of one batch: a CTA costs its per-tree
+// setup (schedule compaction, tables: ~MPCGS_SETUP batches) plus its batches;
+// the launch takes ceil(CTAs / resident CTAs) waves of one CTA (up to four waves),
+// else total work / resident CTAs plus half a CTA of tail.  Few batches per tree and many trees -> one CTA per tree (the setup is
+// not repeated per tile); few trees -> more tiles for parallelism.  Depends only
+// on n, L and the GLOBAL tree count, so every rank tiles (and sums) a proposal's
+// sites identically (world-size invariance).
 #ifndef MPCGS_MAXPER
 #define MPCGS_MAXPER 32
 #endif
+#ifndef MPCGS_SETUP
+#define MPCGS_SETUP 3.0
+#endif
 void prune_tiling(int n, int L, int ntrees_global, int precision, int& tiles, int& sites_per_cta) {
+    const int batch = prune_batch_sites(n, precision);
+    const long batches = (L + batch - 1) / batch;
+    const double slots = 148.0 * (precision == 32 ? 4.0 : 3.0);  // resident CTAs (occupancy of the table kernel)
+    double best = 1e300;
+    int bp = 1;
+    for (int per = 1; per <= MPCGS_MAXPER; ++per) {
+        const long t = (batches + per - 1) / per;
+        const double len = MPCGS_SETUP + (double)std::min<long>(per, batches);
+        const double ctas = (double)ntrees_global * (double)t;
+        const double work = (double)ntrees_global * ((double)t * MPCGS_SETUP + (double)batches);
+        // a few waves: equal CTAs run in lock-step waves; many: the tail averages out
+        const double cost = ctas <= 4.0 * slots ? std::ceil(ctas / slots) * len : work / slots + 0.5 * len;
+        if (cost < best * (1.0 - 1e-9)) {
+            best = cost;
+            bp = per;
+        }
+        if (per >= batches) break;
+    }
+    sites_per_cta = bp * batch;
+    tiles = (L + sites_per_cta - 1) / sites_per_cta;
+}
+
+// incremental rescoring (no per-CTA table setup): as many batches per CTA as
+// keep >= ~8 CTAs per SM busy, up to MPCGS_MAXPER; global N (world-size invariance)
+void incr_tiling(int n, int L, int ntrees_global, int precision, int& tiles, int& sites_per_cta) {
     const int batch = prune_batch_sites(n, precision);
     const long batches = (L + batch - 1) / batch;
     const long want = (long)148 * 8;
@@ -596,8 +628,7 @@ mpcgs_status step_local_launch(mpcgs_ctx* c, uint64_t seed, int64_t step, int N,
     if (c->incremental) {
         IncrArgs ia{};
         ia.count = count;
-        ia.tiles = a.tiles;
-        ia.sites_per_cta = a.sites_per_cta;
+        incr_tiling(c->n, c->L, N, c->precision, ia.tiles, ia.sites_per_cta);
         ia.tile_part = c->s.tile_part;
         ia.tile_cnt = c->s.tile_cnt;
         ia.out = c->s.rec;

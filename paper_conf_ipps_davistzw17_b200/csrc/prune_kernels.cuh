@@ -1021,23 +1021,38 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
     int nops_run = nops_c;
     if constexpr (PT && MPCGS_FUSE_SS) {
         __syncthreads();
-        if (tid == 0) {
-            int j = 0;
-            for (int i = 0; i < nops_c; ++i) {
-                OpRec<T> o = s_opc[i];
-                const uint32_t ty = o.h.x & 3u;
-                if ((ty == OP_TT || ty == OP_TTT) && !(o.h.y & TAB_CHECK) && i + 1 < nops_c &&
-                    (s_opc[i + 1].h.x & 3u) == OP_SS) {
-                    const OpRec<T> ss = s_opc[i + 1];
-                    o.h.x = (o.h.x & ~(3u | OP_CHECK | (3u << OP_FUSED_SHIFT))) | OP_TS | (ss.h.x & OP_CHECK) |
-                            ((ty == OP_TTT ? 2u : 1u) << OP_FUSED_SHIFT);
-                    o.up[0] = ss.up[0];
-                    o.up[1] = ss.up[1];
-                    ++i;
+        if (tid < 32) {  // warp 0: ballot compaction, in place (every write index <= its read index)
+            uint32_t c_keep = 0;
+            bool carry = false;
+            for (int base = 0; base < nops_c; base += 32) {
+                const int i = base + tid;
+                OpRec<T> o;
+                bool head = false;
+                if (i < nops_c) {
+                    o = s_opc[i];
+                    const uint32_t ty = o.h.x & 3u;
+                    head = (ty == OP_TT || ty == OP_TTT) && !(o.h.y & TAB_CHECK) && i + 1 < nops_c &&
+                           (s_opc[i + 1].h.x & 3u) == OP_SS;
+                    if (head) {
+                        const OpRec<T> ss = s_opc[i + 1];
+                        o.h.x = (o.h.x & ~(3u | OP_CHECK | (3u << OP_FUSED_SHIFT))) | OP_TS | (ss.h.x & OP_CHECK) |
+                                ((ty == OP_TTT ? 2u : 1u) << OP_FUSED_SHIFT);
+                        o.up[0] = ss.up[0];
+                        o.up[1] = ss.up[1];
+                    }
                 }
-                s_opc[j++] = o;
+                const unsigned mh = __ballot_sync(0xffffffffu, head);
+                const bool tail = tid == 0 ? carry : ((mh >> (tid - 1)) & 1u) != 0u;
+                const bool keep = i < nops_c && !tail;
+                const unsigned mk = __ballot_sync(0xffffffffu, keep);
+                const uint32_t j = c_keep + __popc(mk & ((1u << tid) - 1u));
+                __syncwarp();
+                if (keep) s_opc[j] = o;
+                __syncwarp();
+                c_keep += __popc(mk);
+                carry = (mh >> 31) & 1u;
             }
-            s_nc = j;
+            if (tid == 0) s_nc = (int)c_keep;
         }
         __syncthreads();
         nops_run = s_nc;
