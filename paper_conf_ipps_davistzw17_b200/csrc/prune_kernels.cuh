@@ -487,7 +487,7 @@ struct Bounds<float> {
     }
 };
 
-// One thread: s_d[2 op + c] = lower bound of log2 d of child c of original op
+// One warp: s_d[2 op + c] = lower bound of log2 d of child c of original op
 // `op`; lpmin = ilogb(min pi) (the root's Eq. 21 dot product).  Walks the
 // compacted op list s_opc (a fused triplet, type OP_TTT, covers original ops o
 // and o+1) and sets s_chk[i] for the ops to check (merged into OP_CHECK later).
@@ -501,8 +501,10 @@ struct __align__(16) OpRec {
 };
 
 template <typename T>
-__device__ void mark_checks(const OpRec<T>* s_opc, const int* s_d, int* s_bnd, unsigned char* s_chk, int nops_c,
-                            int lpmin) {
+__device__ void mark_checks(const OpRec<T>* s_opc, const int* s_d, unsigned char* s_chk, int nops_c, int lpmin,
+                            int lane) {
+    // one warp: the per-op data are loaded in parallel, lane l keeps the bound of
+    // stack level l in a register, and the walk itself broadcasts op by op
     constexpr int TSX = Traits<T>::TS, FLOOR = Bounds<T>::FLOOR;
     auto dsum = [&](const uint4& o) {
         const int i = (int)o.z;
@@ -511,28 +513,46 @@ __device__ void mark_checks(const OpRec<T>* s_opc, const int* s_d, int* s_bnd, u
         return d;
     };
     int dmax = 0;
-    for (int i = 0; i < nops_c; ++i) dmax = max(dmax, -dsum(s_opc[i].h));
+    for (int i = lane; i < nops_c; i += 32) dmax = max(dmax, -dsum(s_opc[i].h));
+#pragma unroll
+    for (int o = 16; o > 0; o >>= 1) dmax = max(dmax, __shfl_xor_sync(0xffffffffu, dmax, o));
     // stack entries stay >= limit, so an op's product is >= 2 limit - dmax >= FLOOR
     const int x = FLOOR + dmax;
     const int limit = x >= 0 ? (x + 1) / 2 : -((-x) / 2);
     const bool all = limit > -TSX;  // no room between checks (e.g. a zero-length branch): check every op
-    for (int i = 0; i < nops_c; ++i) {
-        const uint4 o = s_opc[i].h;
-        const int ty = (int)(o.x & 3u), sp = (int)((o.x >> 2) & 15u);
-        int b = dsum(o), slot;
-        if (ty == (int)OP_TT || ty == (int)OP_TTT) {
-            slot = sp;
-        } else if (ty == (int)OP_TS) {
-            slot = sp - 1;
-            b += s_bnd[sp - 1];
-        } else {
-            slot = sp - 2;
-            b += s_bnd[sp - 2] + s_bnd[sp - 1];
+    int bnd = 0;                    // bound of stack level `lane`
+    for (int base = 0; base < nops_c; base += 32) {
+        const int i = base + lane;
+        int ty = 0, sp = 0, ds = 0;
+        if (i < nops_c) {
+            const uint4 o = s_opc[i].h;
+            ty = (int)(o.x & 3u);
+            sp = (int)((o.x >> 2) & 15u);
+            ds = dsum(o);
         }
-        const bool chk = all || b < limit || (i == nops_c - 1 && b + lpmin < FLOOR);
-        if (chk) b = -TSX;  // after the check: max >= 2^-TS
-        s_chk[i] = chk;
-        s_bnd[slot] = b;
+        const int cnt = min(32, nops_c - base);
+        bool mine = false;
+        for (int q = 0; q < cnt; ++q) {
+            const int qty = __shfl_sync(0xffffffffu, ty, q), qsp = __shfl_sync(0xffffffffu, sp, q);
+            int b = __shfl_sync(0xffffffffu, ds, q);
+            const int b1 = __shfl_sync(0xffffffffu, bnd, max(qsp - 1, 0));
+            const int b2 = __shfl_sync(0xffffffffu, bnd, max(qsp - 2, 0));
+            int slot;
+            if (qty == (int)OP_TT || qty == (int)OP_TTT) {
+                slot = qsp;
+            } else if (qty == (int)OP_TS) {
+                slot = qsp - 1;
+                b += b1;
+            } else {
+                slot = qsp - 2;
+                b += b2 + b1;
+            }
+            const bool chk = all || b < limit || (base + q == nops_c - 1 && b + lpmin < FLOOR);
+            if (chk) b = -TSX;  // after the check: max >= 2^-TS
+            if (lane == slot) bnd = b;
+            if (lane == q) mine = chk;
+        }
+        if (i < nops_c) s_chk[i] = mine;
     }
 }
 
@@ -759,7 +779,6 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
     int* s_d = reinterpret_cast<int*>(reinterpret_cast<unsigned char*>(s_spill) +
                                       sizeof(T) * (size_t)spill_lv * SI * 4 * PRUNE_THREADS);
     int* s_tl = s_d + align16(sizeof(int) * 2 * (size_t)nops) / sizeof(int);  // original codes, then check flags
-    int* s_bnd = s_tl + align16(sizeof(int) * (size_t)nops) / sizeof(int);
     __shared__ double s_red[PRUNE_THREADS / 32];
     __shared__ bool s_last;
     __shared__ int s_nc;  // compacted op count
@@ -863,10 +882,10 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
     }
     __syncthreads();
     const int nops_c = s_nc;
-    // 3. sparse checks (FP64): one thread walks the bounds while the others build the tables
+    // 3. sparse checks (FP64): warp 1 walks the bounds while the others build the tables
     unsigned char* s_chk = reinterpret_cast<unsigned char*>(s_tl);  // s_code is dead after the scan
     if constexpr (sparse_checks<T>()) {
-        if (tid == 32) mark_checks<T>(s_opc, s_d, s_bnd, s_chk, nops_c, Bounds<T>::ilogb(pimin));
+        if (tid >= 32 && tid < 64) mark_checks<T>(s_opc, s_d, s_chk, nops_c, Bounds<T>::ilogb(pimin), tid - 32);
     }
     //    up branch of every op: the child branch its consumer (the first later op
     //    that pops the level it pushes) applies to it -- side a of an SS for the
