@@ -992,7 +992,9 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
         }
     }
     __syncthreads();
-    if constexpr (sparse_checks<T>()) {  // merge the flags (ordered before the op loop by the batch barrier)
+    // the check flags are merged into the op codes after the fold pass (which reads
+    // the codes): by the fusion warp below, or by this loop when there is no fusion
+    if constexpr (sparse_checks<T>() && !(PT && MPCGS_FUSE_SS)) {  // ordered before the op loop by the batch barrier
         for (int op = tid; op < nops_c; op += PRUNE_THREADS)
             if (s_chk[op]) s_opc[op].h.x |= OP_CHECK;
     }
@@ -1049,12 +1051,14 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
                 bool head = false;
                 if (i < nops_c) {
                     o = s_opc[i];
+                    if (sparse_checks<T>() && s_chk[i]) o.h.x |= OP_CHECK;  // the bound walk's flags (S5)
                     const uint32_t ty = o.h.x & 3u;
                     head = (ty == OP_TT || ty == OP_TTT) && !(o.h.y & TAB_CHECK) && i + 1 < nops_c &&
                            (s_opc[i + 1].h.x & 3u) == OP_SS;
                     if (head) {
                         const OpRec<T> ss = s_opc[i + 1];
-                        o.h.x = (o.h.x & ~(3u | OP_CHECK | (3u << OP_FUSED_SHIFT))) | OP_TS | (ss.h.x & OP_CHECK) |
+                        const uint32_t ss_chk = (!sparse_checks<T>() || s_chk[i + 1]) ? OP_CHECK : 0u;
+                        o.h.x = (o.h.x & ~(3u | OP_CHECK | (3u << OP_FUSED_SHIFT))) | OP_TS | ss_chk |
                                 ((ty == OP_TTT ? 2u : 1u) << OP_FUSED_SHIFT);
                         o.up[0] = ss.up[0];
                         o.up[1] = ss.up[1];
