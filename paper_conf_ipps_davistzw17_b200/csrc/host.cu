@@ -11,6 +11,8 @@
 #include <nccl.h>
 
 #include <algorithm>
+#include <chrono>
+#include <thread>
 #include <cmath>
 #include <cstdio>
 #include <cstdlib>
@@ -373,6 +375,23 @@ double host_S(int n, const double* age) {
 
 // A, C, G, T -> 0..3 (S2).  With ambiguity codes (f4, S24): IUPAC letters, '-'
 // and '?' -> 16 + base-set mask (bit X = base X), else -1.
+// fn(i) for i in [0, n), rows spread over up to 32 host threads (alignment ingestion)
+template <typename F>
+void parallel_rows(int n, F&& fn) {
+    const unsigned hw = std::max(1u, std::thread::hardware_concurrency());
+    const int nt = (int)std::min<unsigned>({hw, 32u, (unsigned)std::max(1, n)});
+    if (nt <= 1) {
+        for (int i = 0; i < n; ++i) fn(i);
+        return;
+    }
+    std::vector<std::thread> th;
+    for (int t = 0; t < nt; ++t)
+        th.emplace_back([&, t] {
+            for (int i = t; i < n; i += nt) fn(i);
+        });
+    for (auto& x : th) x.join();
+}
+
 int code_of(char ch, bool ambiguity = false) {
     switch (ch) {
         case 'A': case 'a': return 0;
@@ -815,7 +834,19 @@ mpcgs_status mpcgs_nccl_unique_id(void* out128) {
     return MPCGS_OK;
 }
 
+struct InitTrace {  // MPCGS_TRACE_INIT=1: wall-clock phases of mpcgs_init on stderr
+    bool on = std::getenv("MPCGS_TRACE_INIT") != nullptr;
+    std::chrono::steady_clock::time_point t = std::chrono::steady_clock::now();
+    void mark(const char* what) {
+        if (!on) return;
+        const auto now = std::chrono::steady_clock::now();
+        std::fprintf(stderr, "mpcgs_init %-22s %8.2f ms\n", what, std::chrono::duration<double, std::milli>(now - t).count());
+        t = now;
+    }
+};
+
 mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, double theta0, mpcgs_ctx** out) {
+    InitTrace tr;
     if (!out) return MPCGS_E_ARG;
     *out = nullptr;
     if (!aln || !cfg || !aln->rows) return MPCGS_E_ARG;
@@ -826,17 +857,35 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
     if (cfg->max_proposals < 1 || cfg->max_proposals > MPCGS_MAX_PROPOSALS || cfg->max_samples < 0) return MPCGS_E_ARG;
     if (cfg->world < 1 || cfg->rank < 0 || cfg->rank >= cfg->world || cfg->burnin_steps < 0) return MPCGS_E_ARG;
     // alignment -> codes (S2: ACGT only; with cfg->ambiguity also IUPAC sets, S24)
+    for (int i = 0; i < n; ++i)
+        if (!aln->rows[i]) return MPCGS_E_ARG;
     std::vector<uint8_t> codes((size_t)n * L);
+    // one table lookup per character, rows in parallel; base counts per row for pi (S1)
+    int8_t lut[256];
+    for (int ch = 0; ch < 256; ++ch) lut[ch] = (int8_t)code_of((char)ch, cfg->ambiguity != 0);
+    std::vector<double> row_cnt((size_t)n * 4, 0.0);
+    std::vector<uint8_t> row_bad(n, 0), row_amb(n, 0);
+    parallel_rows(n, [&](int i) {
+        const unsigned char* src = reinterpret_cast<const unsigned char*>(aln->rows[i]);
+        uint8_t* dst = codes.data() + (size_t)i * L;
+        long cnt[4] = {0, 0, 0, 0};
+        int8_t worst = 0;
+        for (int s = 0; s < L; ++s) {
+            const int8_t cd = lut[src[s]];
+            worst = cd < worst ? cd : worst;
+            dst[s] = (uint8_t)cd;
+            if (cd >= 0 && cd < 4) ++cnt[cd];
+            else if (cd >= 16) row_amb[i] = 1;
+        }
+        row_bad[i] = worst < 0;
+        for (int x = 0; x < 4; ++x) row_cnt[(size_t)i * 4 + x] = (double)cnt[x];
+    });
     bool any_amb = false;
     for (int i = 0; i < n; ++i) {
-        if (!aln->rows[i]) return MPCGS_E_ARG;
-        for (int s = 0; s < L; ++s) {
-            int cd = code_of(aln->rows[i][s], cfg->ambiguity != 0);
-            if (cd < 0) return MPCGS_E_ALIGNMENT;
-            codes[(size_t)i * L + s] = (uint8_t)cd;
-            any_amb |= cd >= 16;
-        }
+        if (row_bad[i]) return MPCGS_E_ALIGNMENT;
+        any_amb |= row_amb[i] != 0;
     }
+    tr.mark("codes");
     mpcgs_ctx* c = new mpcgs_ctx();
     c->n = n;
     c->L = L;
@@ -857,9 +906,12 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
     bool emp = false;
     for (int i = 0; i < 4; ++i) emp |= cfg->base_freq[i] < 0.0;
     if (emp) {
-        double cnt[4] = {0, 0, 0, 0}, known = 0.0;
-        for (uint8_t x : codes)
-            if (x < 4) { cnt[x] += 1.0; known += 1.0; }  // ambiguity codes not counted (S24)
+        double cnt[4] = {0, 0, 0, 0}, known = 0.0;  // ambiguity codes not counted (S24)
+        for (int i = 0; i < n; ++i)
+            for (int x = 0; x < 4; ++x) {
+                cnt[x] += row_cnt[(size_t)i * 4 + x];
+                known += row_cnt[(size_t)i * 4 + x];
+            }
         for (int i = 0; i < 4; ++i) pi[i] = known > 0.0 ? cnt[i] / known : 0.25;
     } else {
         double sum = 0.0;
@@ -933,6 +985,7 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
     c->Lpad = (L + 15) & ~15;
     c->incremental = cfg->incremental != 0;
     Layout y = layout(n, Ls, c->Nmax, c->Mmax, c->precision, c->incremental, c->model);
+    tr.mark("model, G0, layout");
     mpcgs_status st = MPCGS_OK;
     do {
         if (cudaStreamCreateWithFlags(&c->work, cudaStreamNonBlocking) != cudaSuccess ||
@@ -956,6 +1009,7 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
             c->own_ws = true;
             c->ws_bytes = y.total;
         }
+        tr.mark("stream, workspace");
         char* b = (char*)c->ws;
         DevState& s = c->s;
         s.n = n; s.nn = c->nn; s.L = L; s.Lpad = c->Lpad; s.nops = c->nops; s.precision = c->precision;
@@ -1017,23 +1071,22 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
         s.site_w = cfg->compress_patterns ? (const double*)(b + y.site_w) : nullptr;
         if ((st = enter(c))) break;
         if (cudaMemsetAsync(c->ws, 0, y.total, c->work) != cudaSuccess) { st = fail(c, MPCGS_E_CUDA, "memset"); break; }
+        tr.mark("enter, memset");
         std::vector<uint8_t> padded((size_t)n * c->Lpad, 0);
-        // byte codes: bases 0..3, or base-set masks 1..15 when the data hold ambiguity codes
-        for (int i = 0; i < n; ++i)
-            for (int site = 0; site < L; ++site) {
-                const int cd = codes[(size_t)i * L + site];
-                padded[(size_t)i * c->Lpad + site] = (uint8_t)(any_amb ? base_set(cd) : cd);
-            }
         const int W2 = codes2_words(L);
         const int si2 = prune_batch_sites(n, c->precision) / PRUNE_THREADS;  // sites per thread of the table kernel
         std::vector<uint32_t> packed((size_t)n * W2, 0u);
-        if (!any_amb)
-            for (int i = 0; i < n; ++i)
-                for (int site = 0; site < L; ++site) {  // thread-interleaved order of the table kernel (Codes)
-                    const int s16 = site & 15, q = s16 / si2, k = s16 % si2;
-                    packed[(size_t)i * W2 + (site >> 4)] |= (uint32_t)codes[(size_t)i * L + site]
-                                                            << ((32 / si2) * k + 2 * q);
-                }
+        int shift[16];  // thread-interleaved order of the table kernel (Codes): site k of thread q
+        for (int s16 = 0; s16 < 16; ++s16) shift[s16] = (32 / si2) * (s16 % si2) + 2 * (s16 / si2);
+        parallel_rows(n, [&](int i) {
+            const uint8_t* src = codes.data() + (size_t)i * L;
+            uint8_t* pb = padded.data() + (size_t)i * c->Lpad;
+            // byte codes: bases 0..3, or base-set masks 1..15 when the data hold ambiguity codes
+            for (int site = 0; site < L; ++site) pb[site] = (uint8_t)(any_amb ? base_set(src[site]) : src[site]);
+            if (any_amb) return;
+            uint32_t* pw = packed.data() + (size_t)i * W2;
+            for (int site = 0; site < L; ++site) pw[site >> 4] |= (uint32_t)src[site] << shift[site & 15];
+        });
         if (cudaMemcpyAsync((void*)s.codes, padded.data(), padded.size(), cudaMemcpyHostToDevice, c->work) != cudaSuccess ||
             (c->codes2 &&
              cudaMemcpyAsync(c->codes2, packed.data(), packed.size() * 4, cudaMemcpyHostToDevice, c->work) != cudaSuccess)) {
@@ -1049,7 +1102,9 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
             st = fail(c, MPCGS_E_CUDA, "pattern weights upload");
             break;
         }
+        tr.mark("pack, upload");
         if ((st = upload_state(c, parent.data(), age.data()))) break;
+        tr.mark("upload_state (G0 score)");
         if (cfg->nccl_id) {  // without an id: no communicator (host-staged exchange when world > 1)
             NcclApi& api = nccl();
             if (!api.ok) { st = fail(c, MPCGS_E_NCCL, "NCCL (libnccl.so.2) could not be loaded"); break; }
@@ -1059,6 +1114,7 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
             if (r != ncclSuccess) { st = fail(c, MPCGS_E_NCCL, "ncclCommInitRank failed"); break; }
         }
         st = leave(c);
+        tr.mark("nccl, leave");
     } while (0);
     if (st != MPCGS_OK) {
         // keep the context so that mpcgs_last_error can explain; caller frees it
