@@ -356,7 +356,9 @@ def main():
     pk, mhz, mp = peaks()
     local_trees = N // world
     gm = args.model != "F81"
-    flops_launch = local_trees * L * (flops_per_site_gm(n) if gm else flops_per_site(n))
+    # the sites the kernel actually scores: all L columns, or the distinct ones under --compress
+    L_scored = ctx.mpcgs_num_patterns() if args.compress else L
+    flops_launch = local_trees * L_scored * (flops_per_site_gm(n) if gm else flops_per_site(n))
     prune_avg_s = (prune_ms / 1e3) / args.steps
     achieved = flops_launch / prune_avg_s / 1e12
     roof = {"bound": "alu", "achieved": achieved, "peak": pk[args.precision], "unit": "TFLOP/s",
@@ -369,6 +371,11 @@ def main():
                            f"{mhz:.0f} MHz (MEASURED_PEAKS sm_max_mhz)",
             "partials_per_s_prune_only": N * L * (n - 1) / (prune_avg_s * world) if world == 1 else
             local_trees * L * (n - 1) / prune_avg_s}
+    if args.compress:
+        roof["traffic"] = None  # the ncu traffic on file is the uncompressed launch's
+        roof["scored_sites"] = L_scored
+        roof["note"] = ("roofline on the distinct columns the kernel scores; value counts all L columns "
+                        "(site-pattern compression, SURVEY 8(f) f3)")
     if args.incremental:
         # k_score_incr recomputes 2 + depth(A) nodes per proposal and site, not n - 1: the
         # full-pruning flop count would overstate its work, so no fraction is claimed here
