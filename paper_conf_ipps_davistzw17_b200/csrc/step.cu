@@ -673,12 +673,15 @@ cudaError_t launch_propose(const DevState& s, uint64_t seed, int64_t step, int s
 }
 
 // ------------------------------------------------------------------ k_draw
-__global__ void __launch_bounds__(DRAW_THREADS) k_draw(DevState s, uint64_t seed, int64_t step_arg, int N,
+// NT threads: 1024, or 128 when N <= 256 (fewer warps at every barrier of a
+// latency-bound step; the weights are then a few per thread)
+template <int NT>
+__global__ void __launch_bounds__(NT) k_draw(DevState s, uint64_t seed, int64_t step_arg, int N,
                                                        int K_arg, int burnin, int64_t M, int64_t total_steps) {
     extern __shared__ __align__(16) double dsm[];
     MPCGS_TS(0);
     double* sC = dsm;  // [N+1] cumulative weights
-    __shared__ double s_red[DRAW_THREADS / 32];
+    __shared__ double s_red[NT / 32];
     __shared__ double s_max;
     __shared__ int s_K, s_store;
     const int tid = threadIdx.x, lane = tid & 31, wid = tid >> 5;
@@ -694,7 +697,7 @@ __global__ void __launch_bounds__(DRAW_THREADS) k_draw(DevState s, uint64_t seed
         r0[3] = s.age[Par];
         r0[4] = -1.0;  // read back only after later barriers
     }
-    const int chunk = (nslots + DRAW_THREADS - 1) / DRAW_THREADS;
+    const int chunk = (nslots + NT - 1) / NT;
     const int i0 = tid * chunk, i1 = min(nslots, i0 + chunk);
     double mx = -CUDART_INF;
     for (int i = i0; i < i1; ++i) mx = fmax(mx, i == 0 ? s.gen[0] : s.rec[(size_t)i * REC]);
@@ -704,7 +707,7 @@ __global__ void __launch_bounds__(DRAW_THREADS) k_draw(DevState s, uint64_t seed
     __syncthreads();
     if (tid == 0) {
         double m2 = -CUDART_INF;
-        for (int w = 0; w < DRAW_THREADS / 32; ++w) m2 = fmax(m2, s_red[w]);
+        for (int w = 0; w < NT / 32; ++w) m2 = fmax(m2, s_red[w]);
         s_max = m2;
         int K;
         int store;
@@ -748,13 +751,13 @@ __global__ void __launch_bounds__(DRAW_THREADS) k_draw(DevState s, uint64_t seed
     if (lane == 31) s_red[wid] = x;
     __syncthreads();
     if (wid == 0) {
-        double v = s_red[lane];
+        double v = lane < NT / 32 ? s_red[lane] : 0.0;
 #pragma unroll
         for (int o = 1; o < 32; o <<= 1) {
             double y = __shfl_up_sync(0xffffffffu, v, o);
             if (lane >= o) v += y;
         }
-        s_red[lane] = v;
+        if (lane < NT / 32) s_red[lane] = v;
     }
     __syncthreads();
     const double before = (wid > 0 ? s_red[wid - 1] : 0.0) + (x - run);
@@ -764,7 +767,7 @@ __global__ void __launch_bounds__(DRAW_THREADS) k_draw(DevState s, uint64_t seed
     const int K = s_K;
     const double total = sC[N];
     const int64_t stored = s.counters[1];
-    for (int d = tid; d < K; d += DRAW_THREADS) {
+    for (int d = tid; d < K; d += NT) {
         const double u = uniform_at(seed, 0u, (uint32_t)step, TAG_DRAW, (uint32_t)d);
         const double xd = u * total;
         int lo = 0, hi = N;  // lowest i with C_i >= x (L1140-1144)
@@ -836,7 +839,7 @@ __global__ void __launch_bounds__(DRAW_THREADS) k_draw(DevState s, uint64_t seed
     if (K_arg < 0 && step + 1 < total_steps) {
         __syncthreads();
         MPCGS_TS(4);
-        context_body<DRAW_THREADS>(s, seed, step + 1, dsm);
+        context_body<NT>(s, seed, step + 1, dsm);
         MPCGS_TS(11);
 #ifdef MPCGS_TIMESTAMPS
         if (threadIdx.x == 0 && step == 2)
@@ -852,11 +855,14 @@ cudaError_t launch_draw(const DevState& s, uint64_t seed, int64_t step, int N, i
     const size_t smem = std::max(sizeof(double) * (size_t)(N + 1), context_smem_bytes(s.n));
     static size_t attr_bytes = 48 * 1024;
     if (smem > attr_bytes) {
-        cudaError_t e = cudaFuncSetAttribute(k_draw, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+        cudaError_t e = cudaFuncSetAttribute(k_draw<128>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+        if (e == cudaSuccess)
+            e = cudaFuncSetAttribute(k_draw<DRAW_THREADS>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
         if (e != cudaSuccess) return e;
         attr_bytes = smem;
     }
-    k_draw<<<1, DRAW_THREADS, smem, st>>>(s, seed, step, N, K, burnin, M, total_steps);
+    if (N <= 256) k_draw<128><<<1, 128, smem, st>>>(s, seed, step, N, K, burnin, M, total_steps);
+    else k_draw<DRAW_THREADS><<<1, DRAW_THREADS, smem, st>>>(s, seed, step, N, K, burnin, M, total_steps);
     return cudaGetLastError();
 }
 
