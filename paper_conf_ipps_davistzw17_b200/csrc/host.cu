@@ -834,6 +834,17 @@ mpcgs_status mpcgs_nccl_unique_id(void* out128) {
     return MPCGS_OK;
 }
 
+// byte codes [n][Lpad] of the flat kernel from the thread-interleaved 2-bit words
+// (site k of thread q of a 16-site word at bit (32/si) k + 2 q); padding stays 0
+__global__ void k_unpack_codes(const uint32_t* __restrict__ codes2, int W2, int n, int L, int Lpad, int si,
+                               uint8_t* __restrict__ out) {
+    const long t = (long)blockIdx.x * blockDim.x + threadIdx.x;
+    if (t >= (long)n * L) return;
+    const int i = (int)(t / L), site = (int)(t - (long)i * L), s16 = site & 15;
+    const int shift = (32 / si) * (s16 % si) + 2 * (s16 / si);
+    out[(size_t)i * Lpad + site] = (uint8_t)((codes2[(size_t)i * W2 + (site >> 4)] >> shift) & 3u);
+}
+
 struct InitTrace {  // MPCGS_TRACE_INIT=1: wall-clock phases of mpcgs_init on stderr
     bool on = std::getenv("MPCGS_TRACE_INIT") != nullptr;
     std::chrono::steady_clock::time_point t = std::chrono::steady_clock::now();
@@ -1072,7 +1083,9 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
         if ((st = enter(c))) break;
         if (cudaMemsetAsync(c->ws, 0, y.total, c->work) != cudaSuccess) { st = fail(c, MPCGS_E_CUDA, "memset"); break; }
         tr.mark("enter, memset");
-        std::vector<uint8_t> padded((size_t)n * c->Lpad, 0);
+        // byte codes (the flat kernel) are unpacked on the device from the 2-bit words
+        // unless the data hold ambiguity codes (then they are the only codes)
+        std::vector<uint8_t> padded(any_amb ? (size_t)n * c->Lpad : 0, 0);
         const int W2 = codes2_words(L);
         const int si2 = prune_batch_sites(n, c->precision) / PRUNE_THREADS;  // sites per thread of the table kernel
         std::vector<uint32_t> packed((size_t)n * W2, 0u);
@@ -1080,18 +1093,29 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
         for (int s16 = 0; s16 < 16; ++s16) shift[s16] = (32 / si2) * (s16 % si2) + 2 * (s16 / si2);
         parallel_rows(n, [&](int i) {
             const uint8_t* src = codes.data() + (size_t)i * L;
-            uint8_t* pb = padded.data() + (size_t)i * c->Lpad;
-            // byte codes: bases 0..3, or base-set masks 1..15 when the data hold ambiguity codes
-            for (int site = 0; site < L; ++site) pb[site] = (uint8_t)(any_amb ? base_set(src[site]) : src[site]);
-            if (any_amb) return;
+            if (any_amb) {  // byte codes: base-set masks 1..15
+                uint8_t* pb = padded.data() + (size_t)i * c->Lpad;
+                for (int site = 0; site < L; ++site) pb[site] = (uint8_t)base_set(src[site]);
+                return;
+            }
             uint32_t* pw = packed.data() + (size_t)i * W2;
             for (int site = 0; site < L; ++site) pw[site >> 4] |= (uint32_t)src[site] << shift[site & 15];
         });
-        if (cudaMemcpyAsync((void*)s.codes, padded.data(), padded.size(), cudaMemcpyHostToDevice, c->work) != cudaSuccess ||
+        if ((any_amb &&
+             cudaMemcpyAsync((void*)s.codes, padded.data(), padded.size(), cudaMemcpyHostToDevice, c->work) != cudaSuccess) ||
             (c->codes2 &&
              cudaMemcpyAsync(c->codes2, packed.data(), packed.size() * 4, cudaMemcpyHostToDevice, c->work) != cudaSuccess)) {
             st = fail(c, MPCGS_E_CUDA, "codes upload");
             break;
+        }
+        if (!any_amb) {
+            const long total = (long)n * L;
+            k_unpack_codes<<<(unsigned)((total + 255) / 256), 256, 0, c->work>>>(c->codes2, W2, n, L, c->Lpad, si2,
+                                                                                 const_cast<uint8_t*>(s.codes));
+            if (cudaGetLastError() != cudaSuccess) {
+                st = fail(c, MPCGS_E_CUDA, "codes unpack");
+                break;
+            }
         }
         if (s.gm && cudaMemcpyAsync((void*)s.gm, gm, sizeof(gm), cudaMemcpyHostToDevice, c->work) != cudaSuccess) {
             st = fail(c, MPCGS_E_CUDA, "model upload");
