@@ -465,7 +465,7 @@ void upgma(int n, int L, const uint8_t* codes, double theta0, int32_t* parent, d
     }
 }
 
-// Sites per CTA: a multiple of the kernel's site batch (1..MPCGS_MAXPER batches),
+// Sites per CTA: a multiple of the kernel's site batch (1..MPCGS_MAXPER = 64 batches),
 // chosen by a small cost model in units of one batch: a CTA costs its per-tree
 // setup (schedule compaction, tables: ~MPCGS_SETUP batches) plus its batches;
 // the launch takes ceil(CTAs / resident CTAs) waves of one CTA (up to four waves),
@@ -474,7 +474,10 @@ void upgma(int n, int L, const uint8_t* codes, double theta0, int32_t* parent, d
 // on n, L and the GLOBAL tree count, so every rank tiles (and sums) a proposal's
 // sites identically (world-size invariance).
 #ifndef MPCGS_MAXPER
-#define MPCGS_MAXPER 32
+#define MPCGS_MAXPER 64
+#endif
+#ifndef MPCGS_MAXPER_INCR
+#define MPCGS_MAXPER_INCR 32
 #endif
 #ifndef MPCGS_SETUP
 #define MPCGS_SETUP 3.0
@@ -503,12 +506,12 @@ void prune_tiling(int n, int L, int ntrees_global, int precision, int& tiles, in
 }
 
 // incremental rescoring (no per-CTA table setup): as many batches per CTA as
-// keep >= ~8 CTAs per SM busy, up to MPCGS_MAXPER; global N (world-size invariance)
+// keep >= ~8 CTAs per SM busy, up to MPCGS_MAXPER_INCR; global N (world-size invariance)
 void incr_tiling(int n, int L, int ntrees_global, int precision, int& tiles, int& sites_per_cta) {
     const int batch = prune_batch_sites(n, precision);
     const long batches = (L + batch - 1) / batch;
     const long want = (long)148 * 8;
-    const int per = (int)std::max<long>(1, std::min<long>(MPCGS_MAXPER, (ntrees_global * batches) / want));
+    const int per = (int)std::max<long>(1, std::min<long>(MPCGS_MAXPER_INCR, (ntrees_global * batches) / want));
     sites_per_cta = per * batch;
     tiles = (L + sites_per_cta - 1) / sites_per_cta;
 }
