@@ -471,8 +471,13 @@ void upgma(int n, int L, const uint8_t* codes, double theta0, int32_t* parent, d
 // the launch takes ceil(CTAs / resident CTAs) waves of one CTA (up to four waves),
 // else total work / resident CTAs plus half a CTA of tail.  Few batches per tree and many trees -> one CTA per tree (the setup is
 // not repeated per tile); few trees -> more tiles for parallelism.  Depends only
-// on n, L and the GLOBAL tree count, so every rank tiles (and sums) a proposal's
-// sites identically (world-size invariance).
+// on n, L, the GLOBAL tree count and the tiling policy, so every rank tiles (and
+// sums) a proposal's sites identically (world-size invariance, P22).  The policy
+// MPCGS_TILING_WORLD = P (environment, default 1) costs the waves of one rank at
+// world size P (N/P trees): a multi-GPU run sets it to its world size so that
+// each rank's share fills whole waves (results then match any other world size
+// run under the same policy bit for bit, and differ from policy 1 by FP rounding
+// of the site sums only).
 #ifndef MPCGS_MAXPER
 #define MPCGS_MAXPER 64
 #endif
@@ -482,8 +487,18 @@ void upgma(int n, int L, const uint8_t* codes, double theta0, int32_t* parent, d
 #ifndef MPCGS_SETUP
 #define MPCGS_SETUP 3.0
 #endif
+static int tiling_world() {
+    static const int w = [] {
+        const char* e = std::getenv("MPCGS_TILING_WORLD");
+        const int v = e ? std::atoi(e) : 1;
+        return v >= 1 ? v : 1;
+    }();
+    return w;
+}
+
 void prune_tiling(int n, int L, int ntrees_global, int precision, int& tiles, int& sites_per_cta) {
     const int batch = prune_batch_sites(n, precision);
+    const double trees = (double)ntrees_global / (double)tiling_world();  // one rank's share under the policy
     const long batches = (L + batch - 1) / batch;
     const double slots = 148.0 * (precision == 32 ? 4.0 : 3.0);  // resident CTAs (occupancy of the table kernel)
     double best = 1e300;
@@ -491,8 +506,8 @@ void prune_tiling(int n, int L, int ntrees_global, int precision, int& tiles, in
     for (int per = 1; per <= MPCGS_MAXPER; ++per) {
         const long t = (batches + per - 1) / per;
         const double len = MPCGS_SETUP + (double)std::min<long>(per, batches);
-        const double ctas = (double)ntrees_global * (double)t;
-        const double work = (double)ntrees_global * ((double)t * MPCGS_SETUP + (double)batches);
+        const double ctas = trees * (double)t;
+        const double work = trees * ((double)t * MPCGS_SETUP + (double)batches);
         // a few waves: equal CTAs run in lock-step waves; many: the tail averages out
         const double cost = ctas <= 4.0 * slots ? std::ceil(ctas / slots) * len : work / slots + 0.5 * len;
         if (cost < best * (1.0 - 1e-9)) {
