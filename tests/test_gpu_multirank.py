@@ -75,3 +75,18 @@ def test_nccl_path_single_rank_matches(P):
     sa, sb = a.mpcgs_get_samples(), b.mpcgs_get_samples()
     for k in sa:
         assert np.array_equal(sa[k], sb[k]), k
+
+
+@pytest.mark.parametrize("policy", ["1", "8"])
+def test_virtual_ranks_under_tiling_policy(P, policy):
+    """P22 holds under each tiling policy (DESIGN 7): bench.py sets
+    MPCGS_TILING_WORLD to its world size; the library reads it once per process."""
+    import os
+    import subprocess
+    import sys
+
+    root = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+    env = dict(os.environ, MPCGS_TILING_WORLD=policy)
+    r = subprocess.run([sys.executable, os.path.join(root, "tools", "invariance_check.py"), "8", "20000", "64", "3"],
+                       env=env, capture_output=True, text=True, timeout=600)
+    assert r.returncode == 0, r.stdout + r.stderr
