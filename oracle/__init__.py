@@ -87,7 +87,9 @@ def lib():
                                          _i32p, _f64p, _f64p, _f64p, _i32p, _i32p, _i32p, _i32p]
         L.orc_run_chain.argtypes = [c.c_int, c.c_int, _u8p, _f64p, c.c_double, c.c_double,
                                     c.c_int, c.c_int, c.c_int, c.c_uint64, _i32p, _f64p, _f64p,
-                                    _f64p, _i64p, _i32p, _i32p]
+                                    _f64p, _i64p, _i32p, _i32p, _i64p]
+        L.orc_em.argtypes = [c.c_int, c.c_int, _u8p, _f64p, c.c_double, c.c_double, c.c_int, c.c_int,
+                             c.c_int, c.c_uint64, c.c_int, c.c_int, _i32p, _f64p, _f64p, _i64p]
         L.orc_log_rel_likelihood.argtypes = [c.c_int, _f64p, c.c_int, c.c_double, c.c_double]
         L.orc_log_rel_likelihood.restype = c.c_double
         L.orc_weighted_mean_S.argtypes = [c.c_int, _f64p, c.c_double, c.c_double]
@@ -296,9 +298,25 @@ def run_chain(codes, pi, u, theta0, N, burnin, M, seed, parent, age):
     st = np.zeros(M, np.int64)
     sl = np.zeros(M, np.int32)
     nf = np.zeros(1, np.int32)
+    ff = np.zeros(1, np.int64)
     _chk(lib().orc_run_chain(n, L, codes, np.ascontiguousarray(pi, np.float64), float(u), theta0,
-                             N, burnin, M, seed, parent, age, S, logL, st, sl, nf))
-    return dict(S=S, logL=logL, step=st, slot=sl, n_flagged=int(nf[0]), parent=parent, age=age)
+                             N, burnin, M, seed, parent, age, S, logL, st, sl, nf, ff))
+    return dict(S=S, logL=logL, step=st, slot=sl, n_flagged=int(nf[0]), first_flag_step=int(ff[0]),
+                parent=parent, age=age)
+
+
+def em(codes, pi, u, theta0, N, burnin, M, seed, n_iter, parent, age, G=4096):
+    """EM re-drive (Fig. 11): per iteration run_chain(seed + it) -> theta_hat -> theta0.
+    Returns the theta trace, each iteration's first flagged step (-1: none) and the final genealogy."""
+    codes = _codes(codes)
+    parent, age = _tree(parent, age)
+    parent, age = parent.copy(), age.copy()
+    n = (len(parent) + 1) // 2
+    trace = np.zeros(n_iter)
+    ff = np.zeros(n_iter, np.int64)
+    _chk(lib().orc_em(n, codes.shape[1], codes, np.ascontiguousarray(pi, np.float64), float(u), float(theta0), N,
+                      burnin, M, seed, n_iter, G, parent, age, trace, ff))
+    return dict(trace=trace, first_flag_step=ff, parent=parent, age=age)
 
 
 # ---------------------------------------------------------------- MLE

@@ -891,10 +891,17 @@ int orc_gmh_step_model(int model, double kappa, int n, int L, const uint8_t* cod
                          slot_S, slot_t12, slot_pair, slot_flag, draws, draw_flag);
 }
 
+/* Alg. 1 (L911-924) with Fig. 12's burn-in (L1312-1327; S17): burn-in steps draw once
+   and store nothing, sampling steps draw min(N, remaining).  The generator
+   gen_parent/gen_age is advanced in place.  n_flagged counts drawn items that were
+   near a threshold; first_flag_step (nullable) receives the first step in which ANY
+   slot choice or draw was flagged (-1 if none): up to that step the chain is
+   determined by the algorithm, after it by the rounding of one comparison. */
 int orc_run_chain(int n, int L, const uint8_t* codes, const double pi[4], double u,
                   double theta0, int N, int burnin, int M, uint64_t seed,
                   int32_t* gen_parent, double* gen_age, double* S_out, double* logL_out,
-                  int64_t* step_out, int32_t* slot_out, int32_t* n_flagged) {
+                  int64_t* step_out, int32_t* slot_out, int32_t* n_flagged,
+                  int64_t* first_flag_step) {
     double gen_logL = orc_log_likelihood(n, L, codes, gen_parent, gen_age, pi, u, NULL);
     double* slot_logL = (double*)malloc(sizeof(double) * (size_t)(N + 1));
     double* slot_S = (double*)malloc(sizeof(double) * (size_t)(N + 1));
@@ -906,6 +913,7 @@ int orc_run_chain(int n, int L, const uint8_t* codes, const double pi[4], double
     int stored = 0, rc = ORC_OK, d, target;
     uint32_t step = 0;
     *n_flagged = 0;
+    if (first_flag_step) *first_flag_step = -1;
     while (stored < M || (int)step < burnin) {
         int burn = (int)step < burnin;
         int K = burn ? 1 : (M - stored < N ? M - stored : N);
@@ -913,6 +921,12 @@ int orc_run_chain(int n, int L, const uint8_t* codes, const double pi[4], double
                           &gen_logL, &target, slot_logL, slot_S, slot_t12, slot_pair, slot_flag,
                           draws, dflag);
         if (rc != ORC_OK) break;
+        if (first_flag_step && *first_flag_step < 0) {
+            for (d = 0; d < K; ++d)
+                if (dflag[d]) *first_flag_step = step;
+            for (d = 1; d <= N; ++d)
+                if (slot_flag[d]) *first_flag_step = step;
+        }
         for (d = 0; d < K; ++d) {
             if (dflag[d] || slot_flag[draws[d]]) (*n_flagged)++;
             if (burn) continue;
@@ -1021,6 +1035,39 @@ double orc_theta_hat(int M, const double* S, int n, double theta0, int G,
         }
         return 0.5 * (a + b);
     }
+}
+
+/*
+ * EM re-drive of Fig. 11 (L1208-1225) and L791-797: n_iter times
+ * { sample with the driving value theta (Alg. 1 + burn-in, seed + it); theta-hat =
+ * argmax of Eq. 25 over those samples; theta0 <- theta-hat }.  The genealogy carries
+ * over between iterations (gen_parent / gen_age advanced in place); every iteration
+ * restarts its step counter at 0 with its own seed.  theta_trace[it] = that
+ * iteration's estimate; first_flag[it] = orc_run_chain's first flagged step (-1 none).
+ * S_buf: caller scratch of M doubles.
+ */
+int orc_em(int n, int L, const uint8_t* codes, const double pi[4], double u, double theta0,
+           int N, int burnin, int M, uint64_t seed, int n_iter, int G, int32_t* gen_parent,
+           double* gen_age, double* theta_trace, int64_t* first_flag) {
+    double* S = (double*)malloc(sizeof(double) * (size_t)M);
+    double* lL = (double*)malloc(sizeof(double) * (size_t)M);
+    int64_t* st = (int64_t*)malloc(sizeof(int64_t) * (size_t)M);
+    int32_t* sl = (int32_t*)malloc(sizeof(int32_t) * (size_t)M);
+    double theta = theta0;
+    int it, rc = ORC_OK;
+    int32_t nf;
+    for (it = 0; it < n_iter; ++it) {
+        rc = orc_run_chain(n, L, codes, pi, u, theta, N, burnin, M, seed + (uint64_t)it, gen_parent,
+                           gen_age, S, lL, st, sl, &nf, first_flag + it);
+        if (rc != ORC_OK) break;
+        theta = orc_theta_hat(M, S, n, theta, G, NULL, NULL);
+        theta_trace[it] = theta;
+    }
+    free(S);
+    free(lL);
+    free(st);
+    free(sl);
+    return rc;
 }
 
 /*

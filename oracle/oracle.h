@@ -100,7 +100,12 @@ int orc_gmh_step_model(int model, double kappa, int n, int L, const uint8_t* cod
 int orc_run_chain(int n, int L, const uint8_t* codes, const double pi[4], double u,
                   double theta0, int N, int burnin, int M, uint64_t seed,
                   int32_t* gen_parent, double* gen_age, double* S_out, double* logL_out,
-                  int64_t* step_out, int32_t* slot_out, int32_t* n_flagged);
+                  int64_t* step_out, int32_t* slot_out, int32_t* n_flagged,
+                  int64_t* first_flag_step);
+/* EM re-drive (Fig. 11) */
+int orc_em(int n, int L, const uint8_t* codes, const double pi[4], double u, double theta0,
+           int N, int burnin, int M, uint64_t seed, int n_iter, int G, int32_t* gen_parent,
+           double* gen_age, double* theta_trace, int64_t* first_flag);
 
 /* Relative likelihood and MLE (Eq. 25-26; 5.1.5; Alg. 2; reading S20) */
 double orc_log_rel_likelihood(int M, const double* S, int n, double theta0, double theta);

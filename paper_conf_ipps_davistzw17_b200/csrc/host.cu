@@ -1222,7 +1222,7 @@ mpcgs_status sample_begin(mpcgs_ctx* c, int32_t N, int64_t M, uint64_t seed) {
         }
         return MPCGS_OK;
     };
-    if (c->timing & 1) {
+    if ((c->timing & 1) && steps > 0) {
         // device-timed steps: events at step boundaries and around every pruning
         // launch; optional L2 flush between steps, outside the timed intervals
         const size_t need = (size_t)4 * steps;
@@ -1430,15 +1430,25 @@ mpcgs_status mpcgs_step_local(mpcgs_ctx* c, int64_t step, int32_t N, uint64_t se
 mpcgs_status mpcgs_get_records(mpcgs_ctx* c, int32_t first, int32_t count, double* host_rec) {
     CHECK_CTX(c);
     if (first < 0 || count < 0 || first + count > c->Nmax + 1 || (count && !host_rec)) return fail(c, MPCGS_E_ARG, "records range");
-    if (count) CU(cudaMemcpy(host_rec, c->s.rec + (size_t)first * REC, 8 * REC * (size_t)count, cudaMemcpyDeviceToHost));
-    return MPCGS_OK;
+    if (!count) return MPCGS_OK;
+    mpcgs_status st = enter(c);
+    if (st) return st;
+    CU(cudaMemcpyAsync(host_rec, c->s.rec + (size_t)first * REC, 8 * REC * (size_t)count, cudaMemcpyDeviceToHost,
+                       c->work));
+    return leave(c);
 }
 
 mpcgs_status mpcgs_put_records(mpcgs_ctx* c, int32_t first, int32_t count, const double* host_rec) {
     CHECK_CTX(c);
     if (first < 1 || count < 0 || first + count > c->Nmax + 1 || (count && !host_rec)) return fail(c, MPCGS_E_ARG, "records range");
-    if (count) CU(cudaMemcpy(c->s.rec + (size_t)first * REC, host_rec, 8 * REC * (size_t)count, cudaMemcpyHostToDevice));
-    return MPCGS_OK;
+    if (!count) return MPCGS_OK;
+    // on the work stream, ordered after the caller's stream, and complete on return
+    // (a pageable H2D cudaMemcpy may return before the DMA lands)
+    mpcgs_status st = enter(c);
+    if (st) return st;
+    CU(cudaMemcpyAsync(c->s.rec + (size_t)first * REC, host_rec, 8 * REC * (size_t)count, cudaMemcpyHostToDevice,
+                       c->work));
+    return leave(c);
 }
 
 mpcgs_status mpcgs_step_finish(mpcgs_ctx* c, int64_t step, int32_t N, int32_t K, uint64_t seed, int32_t* draws) {

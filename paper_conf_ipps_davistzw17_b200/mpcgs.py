@@ -417,8 +417,9 @@ class Context:
         self._chk(lib().mpcgs_get_model(self.h, _ptr(pi), ctypes.byref(mu)), "get_model")
         return pi, mu.value
 
-    def mpcgs_set_timing(self, on):
-        self._chk(lib().mpcgs_set_timing(self.h, int(bool(on))), "set_timing")
+    def mpcgs_set_timing(self, mode):
+        """mode bit 0: CUDA events per step / kernel; bit 1: 256 MiB L2 flush between steps."""
+        self._chk(lib().mpcgs_set_timing(self.h, int(mode) & 3), "set_timing")
 
     def mpcgs_last_timing(self):
         a, b, c = ctypes.c_double(), ctypes.c_double(), ctypes.c_int64()

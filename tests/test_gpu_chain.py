@@ -1,0 +1,136 @@
+"""The production step loop against the oracle on chains that MOVE (SURVEY 8(a)
+a5, a6, a8; 8(c) c6, P20): ``mpcgs_sample`` (CUDA graph of steps, the generator
+commit and the next step's context computed inside ``k_draw``, the sample store)
+and ``mpcgs_em`` (Fig. 11's re-drive) versus ``orc_run_chain`` / ``orc_em``
+from the same start, seed and driving theta.
+
+Alg. 1 L911-924 and Fig. 12: burn-in steps draw once and store
+nothing, sampling steps draw min(N, remaining), the last draw generates the
+next proposal set.  Equivalence (BASELINE.json north_star): slots and steps
+bit-exact, S_G 1e-12 and ln P(D|G) 1e-9 relative, up to the oracle's first
+flagged step (a slot choice or draw within 1e-9 of a threshold, DESIGN
+"Near-threshold draws"); the final genealogy exact when nothing was flagged.
+Each case asserts that its chain actually moves (proposals accepted, distinct
+S_G), so the commit path is exercised.
+"""
+import numpy as np
+import pytest
+
+import synth
+
+pytestmark = pytest.mark.gpu
+
+
+@pytest.fixture(scope="module")
+def P():
+    import torch
+
+    if not torch.cuda.is_available():
+        pytest.skip("no CUDA device")
+    import paper_conf_ipps_davistzw17_b200 as pkg
+
+    pkg.lib()
+    return pkg
+
+
+# (config, overrides, N, burn-in, M, seed, min accepted fraction)
+CHAINS = {
+    # c1's shape with data at theta_true = 0.1 (the config's theta0 = 0.01 drives it)
+    "c1": ("c1", {"theta_true": 0.1}, 16, 8, 400, None, 0.5),
+    # c2's shape (12 tips, N = 64) on 400 bp from UPGMA at theta0 = 0.01
+    "c2": ("c2", {"L": 400}, 64, 20, 3000, 123, 0.08),
+    # c3's tip count on a ragged 257-site alignment, N = 48
+    "c3": ("c3", {"L": 257, "N": 48}, 48, 10, 1440, 77, 0.05),
+}
+
+
+def _setup(orc, key):
+    name, over, N, B, M, seed, min_move = CHAINS[key]
+    wl = synth.workload(name, **over)
+    codes = wl["codes"]
+    pi = orc.base_freqs(codes)
+    u = orc.default_rate(pi)
+    parent, age = orc.upgma(codes, wl["theta0"])
+    seed = wl["chain_seed"] if seed is None else seed
+    return wl, codes, pi, u, parent, age, N, B, M, seed, min_move
+
+
+def _compare(got, ref, M):
+    ff = ref["first_flag_step"]
+    upto = M if ff < 0 else int(np.searchsorted(ref["step"], ff))  # samples of steps before the flag
+    assert upto >= M // 2, f"oracle flagged step {ff} early: only {upto} of {M} samples comparable"
+    sl = slice(0, upto)
+    assert np.array_equal(got["step"][sl], ref["step"][sl])
+    assert np.array_equal(got["slot"][sl], ref["slot"][sl])
+    assert np.allclose(got["S"][sl], ref["S"][sl], rtol=1e-12, atol=0)
+    assert np.all(np.abs(got["logL"][sl] - ref["logL"][sl]) <= 1e-9 * np.abs(ref["logL"][sl]))
+    return ff < 0
+
+
+@pytest.mark.parametrize("incremental,compress", [(False, False), (True, False), (False, True)])
+@pytest.mark.parametrize("key", ["c1", "c2", "c3"])
+def test_sample_loop_matches_oracle_chain(P, orc, key, incremental, compress):
+    if (incremental or compress) and key != "c2":
+        pytest.skip("scoring variants are checked on the c2 chain")
+    wl, codes, pi, u, parent, age, N, B, M, seed, min_move = _setup(orc, key)
+    ref = orc.run_chain(codes, pi, u, wl["theta0"], N, B, M, seed, parent, age)
+    moved = np.mean(ref["slot"] != 0)
+    assert moved >= min_move and len(np.unique(ref["S"])) >= 20, (moved, len(np.unique(ref["S"])))
+    ctx = P.Context(synth.to_strings(codes), wl["theta0"], init_tree=(parent, age), burnin_steps=B,
+                    max_proposals=N, max_samples=M, incremental=incremental, compress_patterns=compress)
+    ctx.mpcgs_sample(N, M, seed)
+    assert ctx.mpcgs_num_samples() == M
+    got = ctx.mpcgs_get_samples()
+    if _compare(got, ref, M):
+        # the committed generator after the last step is the oracle's
+        gp, ga, gl, gS = ctx.mpcgs_get_state()
+        assert np.array_equal(gp, ref["parent"])
+        assert np.allclose(ga, ref["age"], rtol=0, atol=1e-12 * ref["age"].max())
+        assert abs(gS - orc.coalescent_S(ref["age"], len(codes))) <= 1e-12 * gS
+        want = orc.log_likelihood(codes, ref["parent"], ref["age"], pi, u)
+        assert abs(gl - want) <= 1e-9 * abs(want)
+
+
+def test_sample_loop_timing_mode_same_chain(P, orc):
+    """The device-timed loop (plain launches, events, L2 flush between steps) runs the
+    same chain as the CUDA-graph loop."""
+    wl, codes, pi, u, parent, age, N, B, M, seed, _ = _setup(orc, "c1")
+    out = []
+    for mode in (0, 3):
+        ctx = P.Context(synth.to_strings(codes), wl["theta0"], init_tree=(parent, age), burnin_steps=B,
+                        max_proposals=N, max_samples=M)
+        ctx.mpcgs_set_timing(mode)
+        ctx.mpcgs_sample(N, M, seed)
+        out.append(ctx.mpcgs_get_samples())
+        loop_ms, prune_ms, launches = ctx.mpcgs_last_timing()
+        assert loop_ms > 0 and launches > 0
+        if mode:
+            assert 0 < prune_ms < loop_ms
+    for k in out[0]:
+        assert np.array_equal(out[0][k], out[1][k]), k
+
+
+def test_em_trace_matches_oracle(P, orc):
+    """mpcgs_em (sample -> theta-hat -> theta0, chain carried over)
+    against orc_em from the same start: the theta trace to 1e-6 relative (the
+    north star's theta-hat tolerance) and the final genealogy."""
+    wl = synth.workload("c2", L=400)
+    codes = wl["codes"]
+    pi = orc.base_freqs(codes)
+    u = orc.default_rate(pi)
+    parent, age = orc.upgma(codes, wl["theta0"])
+    N, B, M, seed, iters = 64, 20, 1280, 321, 3
+    ref = orc.em(codes, pi, u, wl["theta0"], N, B, M, seed, iters, parent, age)
+    ctx = P.Context(synth.to_strings(codes), wl["theta0"], init_tree=(parent, age), burnin_steps=B,
+                    max_proposals=N, max_samples=M)
+    trace = ctx.mpcgs_em(iters, N, M, seed, 256)
+    ok = np.flatnonzero(ref["first_flag_step"] >= 0)
+    last = iters if ok.size == 0 else int(ok[0])  # iterations before the first flagged one
+    assert last >= 2, ref["first_flag_step"]
+    assert np.allclose(trace[:last], ref["trace"][:last], rtol=1e-6, atol=0), (trace, ref["trace"])
+    # the re-drive moved theta0 away from 0.01 (the estimates differ between iterations)
+    assert abs(ref["trace"][1] / ref["trace"][0] - 1) > 1e-3
+    if last == iters:
+        gp, ga, _, _ = ctx.mpcgs_get_state()
+        assert np.array_equal(gp, ref["parent"])
+        assert np.allclose(ga, ref["age"], rtol=0, atol=1e-10 * ref["age"].max())

@@ -246,6 +246,12 @@ def _lockstep(P, orc, wl, N, steps, seed, K=None, precision=64, incremental=Fals
         assert np.all(np.abs(tr["logL"][ok] - ref["logL"][ok]) <= LL_TOL[precision] * np.abs(ref["logL"][ok]))
         if precision == 64 and not ref["draw_flag"].any() and ok.all():
             assert np.array_equal(tr["draws"], ref["draws"])
+            # the generator the GPU committed (k_draw: last draw's slot, Fig. 12) is the oracle's
+            gp, ga, g_ll2, g_S2 = ctx.mpcgs_get_state()
+            assert np.array_equal(gp, ref["parent"])
+            assert np.allclose(ga, ref["age"], rtol=0, atol=1e-12 * max(height, ref["age"].max()))
+            assert abs(g_ll2 - ref["gen_logL"]) <= LL_TOL[precision] * abs(ref["gen_logL"])
+            assert abs(g_S2 - ref["S"][ref["draws"][-1]]) <= 1e-12 * abs(g_S2)
         else:
             skipped += 1
         parent, age, gl = ref["parent"], ref["age"], ref["gen_logL"]
@@ -322,26 +328,7 @@ def test_root_case_and_n3(P, orc):
     assert _lockstep(P, orc, wl, 8, 20, 9) <= 1
 
 
-# ------------------------------------------------------------------ free-running chain vs oracle
-def test_free_running_chain_c1(P, orc):
-    wl = synth.workload("c1")
-    codes = wl["codes"]
-    pi = orc.base_freqs(codes)
-    u = orc.default_rate(pi)
-    parent, age = orc.upgma(codes, wl["theta0"])
-    N, M, B = 16, 400, 8
-    ref = orc.run_chain(codes, pi, u, wl["theta0"], N, B, M, wl["chain_seed"], parent, age)
-    ctx = _ctx(P, codes, wl["theta0"], burnin_steps=B, max_proposals=N, max_samples=M)
-    ctx.mpcgs_sample(N, M, wl["chain_seed"])
-    got = ctx.mpcgs_get_samples()
-    assert ctx.mpcgs_num_samples() == M
-    # identical until the first near-threshold flag of the oracle (none expected here)
-    if ref["n_flagged"] == 0:
-        assert np.array_equal(got["slot"], ref["slot"])
-        assert np.array_equal(got["step"], ref["step"])
-        assert np.allclose(got["S"], ref["S"], rtol=1e-11)
-        assert np.all(np.abs(got["logL"] - ref["logL"]) <= 1e-9 * np.abs(ref["logL"]))
-
+# The free-running loop (mpcgs_sample, mpcgs_em) on moving chains: tests/test_gpu_chain.py
 
 # ------------------------------------------------------------------ theta MLE
 def test_theta_hat_matches_oracle(P, orc):
