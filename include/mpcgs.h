@@ -105,6 +105,12 @@ typedef struct {
                               empirical pi counts A/C/G/T only; UPGMA counts a site as a
                               difference when the two sets are disjoint).  0: S2, anything but
                               ACGT -> MPCGS_E_ALIGNMENT */
+    const char* init_newick; /* host, NUL-terminated Newick G0 (the paper's data come
+                              with ms trees, L1499), e.g. "((0:0.1,1:0.1):0.3,2:0.4);": binary,
+                              every branch with a length, tips labelled by row index 0..n-1 and
+                              contemporaneous (S22, to 1e-5 of the height); copied at init.
+                              Takes precedence over init_parent/init_age; NULL -> those or UPGMA.
+                              Parse errors -> MPCGS_E_ARG (mpcgs_last_error says where) */
 } mpcgs_config;
 
 #define MPCGS_MODEL_F81 0
@@ -155,7 +161,9 @@ mpcgs_status mpcgs_sample(mpcgs_ctx* ctx, int32_t n_proposals, int64_t n_samples
 
 /* theta-hat = argmax L(theta) over the stored samples (Eq. 25-26; S20): a log-spaced
  * grid of n_grid points (3..MPCGS_MAX_GRID) over [S_min, S_max]/(n-1) evaluated on
- * the device, then safeguarded Newton on d lnL/d theta inside the best bracket.
+ * the device, then safeguarded Newton on d lnL/d theta inside the grid cells of every
+ * local maximum of the grid curve (up to 4); the refined point of highest ln L wins
+ * (L(theta) can be bimodal).
  * grid_theta / grid_logL: host [n_grid] or NULL; grid_logL = ln L(theta). */
 mpcgs_status mpcgs_estimate_theta(mpcgs_ctx* ctx, double* theta_hat, int32_t n_grid,
                                   double* grid_theta, double* grid_logL);
@@ -201,6 +209,13 @@ mpcgs_status mpcgs_step_finish(mpcgs_ctx* ctx, int64_t step, int32_t n_proposals
  * statistic S_G = sum k(k-1)T_k (Eq. 18), ln P(D|G), step index, slot index. */
 mpcgs_status mpcgs_get_samples(mpcgs_ctx* ctx, int64_t first, int64_t count, double* S,
                                double* logL, int64_t* step, int32_t* slot);
+/* Replace the sample store by `count` given samples (1 <= count <= max_samples):
+ * host S[count] (S_G >= 0, finite) and logL[count] (nullable -> 0), drawn under the
+ * driving value theta0 > 0, for the theta MLE (Eq. 25-26 depend on the samples only
+ * through S_G and theta0).  Step and slot indices read back as -1.  Used to test
+ * mpcgs_estimate_theta on prescribed sample sets (e.g. S20's bimodal case). */
+mpcgs_status mpcgs_load_samples(mpcgs_ctx* ctx, int64_t count, const double* S, const double* logL,
+                                double theta0);
 int64_t mpcgs_num_samples(const mpcgs_ctx* ctx);
 /* Sites the kernels score: distinct columns with compress_patterns, else n_sites. */
 int32_t mpcgs_num_patterns(const mpcgs_ctx* ctx);
@@ -259,6 +274,11 @@ mpcgs_status mpcgs_shard_range(int32_t n_proposals, int32_t rank, int32_t world,
  * mask for an ambiguity code (S24: a site differs when the two sets are disjoint). */
 mpcgs_status mpcgs_upgma(int32_t n_seq, int32_t n_sites, const uint8_t* codes, double theta0,
                          int32_t* parent, double* age);
+/* [host-only] Parse a Newick genealogy of n_seq tips (grammar and rules of
+ * mpcgs_config.init_newick) into parent/age [2n-1] host arrays: interior ids n..2n-2 in
+ * ascending age (ties: post-order), a node's age = its longest path down to a tip.
+ * MPCGS_E_ARG on any syntax / shape / label / ultrametricity error. */
+mpcgs_status mpcgs_parse_newick(int32_t n_seq, const char* newick, int32_t* parent, double* age);
 /* [host-only] Post-order register schedule of a tree as used by the pruning kernel
  * (DESIGN.md "prune"): op[i] = type | sp<<2 | tipA<<6 | tipB<<17, e[2i], e[2i+1] branch
  * factors exp(-u t); returns the register need (max stack depth) or < 0 on error. */

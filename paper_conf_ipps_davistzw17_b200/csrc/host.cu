@@ -307,6 +307,157 @@ int check_tree(int n, const int32_t* parent, const double* age, std::string& why
     return 0;
 }
 
+// Newick G0 (SURVEY 8(b) init_newick; the paper reads its initial genealogy from
+// UPGMA, 5.1.3 L1287-1295, and its test data come with ms's Newick trees, L1499).
+// Grammar: tree := node [':' len] ';'   node := '(' node ',' node ')' [label] | label,
+// each non-root node with ':' length >= 0.  Tip labels are row indices "0".."n-1".
+// Tips are contemporaneous (S22): every tip depth must agree with the deepest to
+// 1e-5 of the height; a node's age is the longest path from it down to a tip, so
+// ages never decrease towards the root.  Interior ids n..2n-2 ascend with age (ties:
+// post-order), the creation order of a coalescent simulation.  0 or -1 with `why`.
+int parse_newick(int n, const char* text, int32_t* parent, double* age, std::string& why) {
+    struct Nd { int par = -1, c0 = -1, c1 = -1, tip = -1; double len = 0.0; };
+    std::vector<Nd> nd;
+    nd.reserve(2 * (size_t)n);
+    const char* p = text;
+    auto ws = [&]() { while (*p == ' ' || *p == '\t' || *p == '\n' || *p == '\r') ++p; };
+    auto label = [&](std::string& out) {
+        out.clear();
+        while (*p && !std::strchr("(),:; \t\r\n", *p)) out.push_back(*p++);
+    };
+    auto number = [&](double& v) -> bool {
+        char* end = nullptr;
+        v = std::strtod(p, &end);
+        if (end == p) return false;
+        p = end;
+        return std::isfinite(v) && v >= 0.0;
+    };
+    std::vector<char> seen(n, 0);
+    std::vector<int> stack;  // open internal nodes
+    int root = -1;
+    std::string lab;
+    // iterative parse: each node is created when first reached
+    auto new_node = [&](int par) {
+        nd.push_back(Nd{});
+        const int id = (int)nd.size() - 1;
+        nd[id].par = par;
+        if (par >= 0) {
+            if (nd[par].c0 < 0) nd[par].c0 = id;
+            else if (nd[par].c1 < 0) nd[par].c1 = id;
+            else return -2;  // multifurcation
+        }
+        return id;
+    };
+    auto parse_len = [&](int id) -> bool {
+        ws();
+        if (*p == ':') {
+            ++p;
+            ws();
+            if (!number(nd[id].len)) return false;
+        } else if (nd[id].par >= 0) {
+            return false;  // every branch needs a length
+        }
+        return true;
+    };
+    ws();
+    int cur_par = -1;
+    for (;;) {
+        ws();
+        if ((int)nd.size() > 2 * n) { why = "more nodes than 2n-1"; return -1; }
+        if (*p == '(') {
+            ++p;
+            const int id = new_node(cur_par);
+            if (id == -2) { why = "a node has more than two children"; return -1; }
+            if (cur_par < 0) root = id;
+            stack.push_back(id);
+            cur_par = id;
+            continue;
+        }
+        // a tip
+        label(lab);
+        if (lab.empty()) { why = std::string("expected a tip label at '") + std::string(p, std::min<size_t>(16, std::strlen(p))) + "'"; return -1; }
+        char* end = nullptr;
+        const long t = std::strtol(lab.c_str(), &end, 10);
+        if (*end || t < 0 || t >= n) { why = "tip label '" + lab + "' is not a row index 0..n-1"; return -1; }
+        if (seen[t]) { why = "tip " + lab + " appears twice"; return -1; }
+        seen[t] = 1;
+        const int id = new_node(cur_par);
+        if (id == -2) { why = "a node has more than two children"; return -1; }
+        if (cur_par < 0) { why = "the tree is a single tip"; return -1; }
+        nd[id].tip = (int)t;
+        if (!parse_len(id)) { why = "tip " + lab + ": missing or invalid branch length"; return -1; }
+        // close groups
+        for (;;) {
+            ws();
+            if (*p == ',') {
+                ++p;
+                break;  // next sibling under cur_par
+            }
+            if (*p == ')') {
+                ++p;
+                const int done = stack.back();
+                stack.pop_back();
+                if (nd[done].c1 < 0) { why = "an internal node has one child"; return -1; }
+                label(lab);  // optional internal label, ignored
+                if (!parse_len(done)) { why = "internal node: missing or invalid branch length"; return -1; }
+                cur_par = stack.empty() ? -1 : stack.back();
+                if (stack.empty()) break;
+                continue;
+            }
+            if (*p == ';' && stack.empty()) break;
+            why = std::string("unexpected character '") + (*p ? *p : '0') + "'";
+            return -1;
+        }
+        if (stack.empty()) break;
+    }
+    ws();
+    if (*p != ';') { why = "missing ';'"; return -1; }
+    if ((int)nd.size() != 2 * n - 1) { why = "the tree must have n tips and n-1 binary internal nodes"; return -1; }
+    for (int t = 0; t < n; ++t)
+        if (!seen[t]) { why = "tip " + std::to_string(t) + " missing"; return -1; }
+    const int m = (int)nd.size();
+    std::vector<double> depth(m, 0.0), h(m, 0.0);
+    for (int v = 0; v < m; ++v)  // parents precede children in creation order
+        if (nd[v].par >= 0) depth[v] = depth[nd[v].par] + nd[v].len;
+    double height = 0.0;
+    for (int v = 0; v < m; ++v)
+        if (nd[v].tip >= 0) height = std::max(height, depth[v]);
+    for (int v = 0; v < m; ++v)
+        if (nd[v].tip >= 0 && height - depth[v] > 1e-5 * height) { why = "tips are not contemporaneous (S22)"; return -1; }
+    // age = longest path down to a tip; children are created after their parent
+    std::vector<int> post;  // post-order (children before parents)
+    {
+        std::vector<std::pair<int, int>> st{{root, 0}};
+        while (!st.empty()) {
+            auto& [v, k] = st.back();
+            if (nd[v].tip < 0 && k < 2) {
+                const int ch = k == 0 ? nd[v].c0 : nd[v].c1;
+                ++k;
+                st.push_back({ch, 0});
+                continue;
+            }
+            post.push_back(v);
+            st.pop_back();
+        }
+    }
+    std::vector<int> interior;
+    for (int v : post) {
+        if (nd[v].tip >= 0) continue;
+        h[v] = std::max(h[nd[v].c0] + nd[nd[v].c0].len, h[nd[v].c1] + nd[nd[v].c1].len);
+        interior.push_back(v);
+    }
+    std::stable_sort(interior.begin(), interior.end(), [&](int a, int b) { return h[a] < h[b]; });
+    std::vector<int> id(m, -1);
+    for (int v = 0; v < m; ++v)
+        if (nd[v].tip >= 0) id[v] = nd[v].tip;
+    for (size_t k = 0; k < interior.size(); ++k) id[interior[k]] = n + (int)k;
+    for (int v = 0; v < m; ++v) {
+        parent[id[v]] = nd[v].par >= 0 ? id[nd[v].par] : -1;
+        age[id[v]] = nd[v].tip >= 0 ? 0.0 : h[v];
+    }
+    return 0;
+}
+
 struct HostTree {
     std::vector<int32_t> left, right, need;
     std::vector<double> e, em;
@@ -779,6 +930,17 @@ int32_t mpcgs_tree_schedule(int32_t n, const int32_t* parent, const double* age,
     return host_schedule<double>(n, ht, op, e);
 }
 
+mpcgs_status mpcgs_parse_newick(int32_t n, const char* newick, int32_t* parent, double* age) {
+    if (n < 2 || n > MPCGS_MAX_SEQ || !newick || !parent || !age) return MPCGS_E_ARG;
+    std::string why;
+    std::vector<int32_t> p(2 * (size_t)n - 1);
+    std::vector<double> a(2 * (size_t)n - 1);
+    if (parse_newick(n, newick, p.data(), a.data(), why) || check_tree(n, p.data(), a.data(), why)) return MPCGS_E_ARG;
+    std::copy(p.begin(), p.end(), parent);
+    std::copy(a.begin(), a.end(), age);
+    return MPCGS_OK;
+}
+
 mpcgs_status mpcgs_phylip_dims(const char* path, int32_t* n_seq, int32_t* n_sites) {
     FILE* f = path ? std::fopen(path, "r") : nullptr;
     if (!f) return MPCGS_E_ALIGNMENT;
@@ -972,7 +1134,15 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
     // G0
     std::vector<int32_t> parent(c->nn);
     std::vector<double> age(c->nn);
-    if (cfg->init_parent && cfg->init_age) {
+    if (cfg->init_newick) {
+        std::string why;
+        if (parse_newick(n, cfg->init_newick, parent.data(), age.data(), why) ||
+            check_tree(n, parent.data(), age.data(), why)) {
+            c->err = "init_newick: " + why;
+            *out = c;
+            return MPCGS_E_ARG;
+        }
+    } else if (cfg->init_parent && cfg->init_age) {
         std::copy(cfg->init_parent, cfg->init_parent + c->nn, parent.begin());
         std::copy(cfg->init_age, cfg->init_age + c->nn, age.begin());
     } else {
@@ -1381,6 +1551,26 @@ mpcgs_status mpcgs_get_samples(mpcgs_ctx* c, int64_t first, int64_t count, doubl
     return MPCGS_OK;
 }
 
+mpcgs_status mpcgs_load_samples(mpcgs_ctx* c, int64_t count, const double* S, const double* logL, double theta0) {
+    CHECK_CTX(c);
+    if (c->pend.active) return fail(c, MPCGS_E_STATE, "a sampling loop is still pending");
+    if (count < 1 || count > c->Mmax || !S) return fail(c, MPCGS_E_ARG, "load_samples: 1 <= count <= max_samples");
+    if (!(theta0 > 0.0) || !std::isfinite(theta0)) return fail(c, MPCGS_E_ARG, "load_samples: theta0 must be positive");
+    for (int64_t i = 0; i < count; ++i)
+        if (!(S[i] >= 0.0) || !std::isfinite(S[i])) return fail(c, MPCGS_E_ARG, "load_samples: S must be finite, >= 0");
+    mpcgs_status st = enter(c);
+    if (st) return st;
+    CU(cudaMemcpyAsync(c->s.sS, S, 8 * (size_t)count, cudaMemcpyHostToDevice, c->work));
+    if (logL) CU(cudaMemcpyAsync(c->s.sL, logL, 8 * (size_t)count, cudaMemcpyHostToDevice, c->work));
+    else CU(cudaMemsetAsync(c->s.sL, 0, 8 * (size_t)count, c->work));
+    CU(cudaMemsetAsync(c->s.sStep, 0xff, 8 * (size_t)count, c->work));
+    CU(cudaMemsetAsync(c->s.sSlot, 0xff, 4 * (size_t)count, c->work));
+    if ((st = leave(c))) return st;
+    c->nsamples = count;
+    c->sample_theta0 = theta0;
+    return MPCGS_OK;
+}
+
 mpcgs_status mpcgs_score_trees(mpcgs_ctx* c, int32_t n_trees, const int32_t* parent, const double* age,
                                double* logL_out) {
     CHECK_CTX(c);
@@ -1627,9 +1817,6 @@ mpcgs_status estimate_theta_impl(mpcgs_ctx* const* cs, int K, double* theta_hat,
         if (h[G + g] > h[G + best]) best = g;
     if (grid_theta) std::copy(h.begin(), h.begin() + G, grid_theta);
     if (grid_logL) std::copy(h.begin() + G, h.end(), grid_logL);
-    double blo = best > 0 ? h[best - 1] : lo, bhi = best < G - 1 ? h[best + 1] : hi;
-    if (best == 0) blo = lo;
-    if (best == G - 1) bhi = hi;
     // f(theta) = sum_l (S_w,l - (n_l - 1) theta) has the sign of d lnL / d theta
     auto f_at = [&](double th, double& f, double& fp) -> mpcgs_status {
         double fs = 0.0, vs = 0.0;
@@ -1646,38 +1833,43 @@ mpcgs_status estimate_theta_impl(mpcgs_ctx* const* cs, int K, double* theta_hat,
         fp = vs / (th * th) - dof;
         return MPCGS_OK;
     };
-    mpcgs_status st;
-    double flo, fhi, dummy;
-    if ((st = f_at(blo, flo, dummy))) return st;
-    if ((st = f_at(bhi, fhi, dummy))) return st;
-    double th = h[best];
-    if (flo >= 0.0 && fhi <= 0.0) {
-        for (int it = 0; it < 200; ++it) {
-            double f, fp;
-            if ((st = f_at(th, f, fp))) return st;
-            if (f >= 0.0) blo = th;
-            else bhi = th;
-            double tn = (fp < 0.0) ? th - f / fp : 0.5 * (blo + bhi);
-            if (!(tn > blo && tn < bhi)) tn = 0.5 * (blo + bhi);
-            if (std::fabs(tn - th) <= 1e-14 * th || bhi - blo <= 1e-15 * bhi) {
-                th = tn;
-                break;
-            }
-            th = tn;
+    // ln L at theta (summed over loci), exact LSE shift
+    auto ll = [&](double t, double& v) -> mpcgs_status {
+        double tot = 0.0;
+        for (int l = 0; l < K; ++l) {
+            double m[4];
+            mpcgs_status s2 = moments(cs[l], t, 0.0, smin[l], smax[l], m);
+            if (s2) return s2;
+            tot += (double)(cs[l]->n - 1) * std::log(cs[l]->sample_theta0 / t) + m[3] + std::log(m[0]);
         }
-    } else {
-        // golden-section search on ln L inside the bracket
-        auto ll = [&](double t, double& v) -> mpcgs_status {
-            double tot = 0.0;
-            for (int l = 0; l < K; ++l) {
-                double m[4];
-                mpcgs_status s2 = moments(cs[l], t, 0.0, smin[l], smax[l], m);
-                if (s2) return s2;
-                tot += (double)(cs[l]->n - 1) * std::log(cs[l]->sample_theta0 / t) + m[3] + std::log(m[0]);
+        v = tot;
+        return MPCGS_OK;
+    };
+    // refine the maximum inside the grid cells around grid point b
+    auto refine = [&](int b, double& th) -> mpcgs_status {
+        mpcgs_status st;
+        double blo = b > 0 ? h[b - 1] : lo, bhi = b < G - 1 ? h[b + 1] : hi;
+        double flo, fhi, dummy;
+        if ((st = f_at(blo, flo, dummy))) return st;
+        if ((st = f_at(bhi, fhi, dummy))) return st;
+        th = h[b];
+        if (flo >= 0.0 && fhi <= 0.0) {  // safeguarded Newton on the stationarity condition
+            for (int it = 0; it < 200; ++it) {
+                double f, fp;
+                if ((st = f_at(th, f, fp))) return st;
+                if (f >= 0.0) blo = th;
+                else bhi = th;
+                double tn = (fp < 0.0) ? th - f / fp : 0.5 * (blo + bhi);
+                if (!(tn > blo && tn < bhi)) tn = 0.5 * (blo + bhi);
+                if (std::fabs(tn - th) <= 1e-14 * th || bhi - blo <= 1e-15 * bhi) {
+                    th = tn;
+                    break;
+                }
+                th = tn;
             }
-            v = tot;
             return MPCGS_OK;
-        };
+        }
+        // golden-section search on ln L inside the bracket
         const double gr = 0.6180339887498949;
         double a = blo, bb = bhi, x1 = bb - gr * (bb - a), x2 = a + gr * (bb - a), v1, v2;
         if ((st = ll(x1, v1)) || (st = ll(x2, v2))) return st;
@@ -1686,6 +1878,34 @@ mpcgs_status estimate_theta_impl(mpcgs_ctx* const* cs, int K, double* theta_hat,
             else { a = x1; x1 = x2; v1 = v2; x2 = a + gr * (bb - a); if ((st = ll(x2, v2))) return st; }
         }
         th = 0.5 * (a + bb);
+        return MPCGS_OK;
+    };
+    // S20: ln L may be bimodal and a coarse grid may rank two close modes wrongly, so
+    // every local maximum of the grid curve (up to 4, highest first) is refined and
+    // the refined point with the highest ln L is theta-hat (the global argmax)
+    std::vector<int> cand;
+    for (int g = 0; g < G; ++g) {
+        const double v = h[G + g];
+        if ((g == 0 || v >= h[G + g - 1]) && (g == G - 1 || v > h[G + g + 1])) cand.push_back(g);
+    }
+    std::sort(cand.begin(), cand.end(), [&](int a, int b) { return h[G + a] > h[G + b]; });
+    if (cand.empty()) cand.push_back(best);
+    if (cand.size() > 4) cand.resize(4);
+    mpcgs_status st;
+    double th = 0.0, th_ll = -INFINITY;
+    for (size_t k = 0; k < cand.size(); ++k) {
+        double t = 0.0;
+        if ((st = refine(cand[k], t))) return st;
+        if (cand.size() == 1) {
+            th = t;
+            break;
+        }
+        double v;
+        if ((st = ll(t, v))) return st;
+        if (v > th_ll) {
+            th_ll = v;
+            th = t;
+        }
     }
     *theta_hat = th;
     return MPCGS_OK;

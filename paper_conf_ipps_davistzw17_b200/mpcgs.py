@@ -40,7 +40,7 @@ class mpcgs_config(ctypes.Structure):
         ("nccl_id", ctypes.c_void_p), ("stream", ctypes.c_void_p), ("workspace", ctypes.c_void_p),
         ("workspace_bytes", ctypes.c_size_t), ("incremental", ctypes.c_int32),
         ("compress_patterns", ctypes.c_int32), ("model", ctypes.c_int32), ("kappa", ctypes.c_double),
-        ("ambiguity", ctypes.c_int32),
+        ("ambiguity", ctypes.c_int32), ("init_newick", ctypes.c_char_p),
     ]
 
 
@@ -73,6 +73,7 @@ _SIGS = {
     "mpcgs_step_finish": (_i32, [_P, _i64, _i32, _i32, _u64, _P]),
     "mpcgs_get_samples": (_i32, [_P, _i64, _i64, _P, _P, _P, _P]),
     "mpcgs_num_samples": (_i64, [_P]),
+    "mpcgs_load_samples": (_i32, [_P, _i64, _P, _P, _f64]),
     "mpcgs_num_patterns": (_i32, [_P]),
     "mpcgs_set_theta0": (_i32, [_P, _f64]),
     "mpcgs_em": (_i32, [_P, _i32, _i32, _i64, _u64, _i32, _P]),
@@ -87,6 +88,7 @@ _SIGS = {
     "mpcgs_shard_range": (_i32, [_i32, _i32, _i32, _P, _P]),
     "mpcgs_upgma": (_i32, [_i32, _i32, _P, _f64, _P, _P]),
     "mpcgs_tree_schedule": (_i32, [_i32, _P, _P, _f64, _P, _P]),
+    "mpcgs_parse_newick": (_i32, [_i32, ctypes.c_char_p, _P, _P]),
     "mpcgs_phylip_dims": (_i32, [ctypes.c_char_p, _P, _P]),
     "mpcgs_phylip_read": (_i32, [ctypes.c_char_p, _P, _i32]),
     "mpcgs_philox": (None, [_P, _P, _P]),
@@ -170,6 +172,15 @@ def mpcgs_tree_schedule(parent, age, mu):
     if d < 0:
         raise MpcgsError(d, "tree_schedule")
     return op, e.reshape(n - 1, 4), d
+
+
+def mpcgs_parse_newick(n_seq, newick):
+    parent = np.zeros(2 * n_seq - 1, np.int32)
+    age = np.zeros(2 * n_seq - 1)
+    st = lib().mpcgs_parse_newick(int(n_seq), newick.encode(), _ptr(parent), _ptr(age))
+    if st:
+        raise MpcgsError(st, "parse_newick")
+    return parent, age
 
 
 def mpcgs_phylip_read(path):
@@ -257,7 +268,7 @@ class Context:
     def __init__(self, rows, theta0, *, precision=64, burnin_steps=0, max_proposals=1024,
                  max_samples=1 << 20, base_freq=None, mu=0.0, init_tree=None, rank=0, world=1,
                  nccl_id=None, stream=None, workspace=None, phylip=None, incremental=False,
-                 compress_patterns=False, model="F81", kappa=0.0, ambiguity=False):
+                 compress_patterns=False, model="F81", kappa=0.0, ambiguity=False, init_newick=None):
         L = lib()
         cfg = mpcgs_config()
         L.mpcgs_config_default(ctypes.byref(cfg))
@@ -275,6 +286,10 @@ class Context:
         cfg.kappa = float(kappa)
         cfg.ambiguity = int(bool(ambiguity))
         self._keep = []
+        if init_newick is not None:
+            nw = init_newick.encode() if isinstance(init_newick, str) else bytes(init_newick)
+            self._keep.append(nw)
+            cfg.init_newick = nw
         if init_tree is not None:
             p = _i32a(init_tree[0])
             a = _f64a(init_tree[1])
@@ -402,6 +417,11 @@ class Context:
         self._chk(lib().mpcgs_get_samples(self.h, first, count, _ptr(S), _ptr(ll), _ptr(st), _ptr(sl)),
                   "get_samples")
         return dict(S=S, logL=ll, step=st, slot=sl)
+
+    def mpcgs_load_samples(self, S, theta0, logL=None):
+        S = _f64a(S)
+        ll = None if logL is None else _f64a(logL, S.size)
+        self._chk(lib().mpcgs_load_samples(self.h, S.size, _ptr(S), _ptr(ll), float(theta0)), "load_samples")
 
     def mpcgs_set_theta0(self, theta0):
         self._chk(lib().mpcgs_set_theta0(self.h, theta0), "set_theta0")

@@ -374,3 +374,29 @@ def test_argument_errors(P):
         ctx.mpcgs_sample(32, 10, 1)       # N above capacity
     with pytest.raises(P.MpcgsError):
         ctx.mpcgs_sample(16, 1000, 1)     # M above capacity
+
+
+def test_init_newick_equals_arrays(P, orc):
+    """SURVEY 8(b) init_newick: a context started from a Newick G0 holds the same
+    generator (and its likelihood) as one started from the parsed arrays."""
+    wl = synth.workload("c2", L=300)
+    codes, p, a = wl["codes"], wl["true_parent"], wl["true_age"]
+    n = len(codes)
+    kids = {v: [] for v in range(2 * n - 1)}
+    for v in range(2 * n - 1):
+        if p[v] >= 0:
+            kids[int(p[v])].append(v)
+
+    def rec(v):
+        return str(v) if v < n else "(" + ",".join(f"{rec(c)}:{float(a[v] - a[c])!r}" for c in kids[v]) + ")"
+
+    nw = rec(int(np.where(p < 0)[0][0])) + ";"
+    c1 = _ctx(P, codes, wl["theta0"], init_newick=nw, max_proposals=8, max_samples=8)
+    g1 = c1.mpcgs_get_state()
+    assert np.array_equal(g1[0], p) and np.allclose(g1[1], a, rtol=1e-13)
+    pi = orc.base_freqs(codes)
+    want = orc.log_likelihood(codes, p, a, pi, orc.default_rate(pi))
+    assert abs(g1[2] - want) <= 1e-9 * abs(want)
+    with pytest.raises(P.MpcgsError) as ei:
+        _ctx(P, codes, wl["theta0"], init_newick="((0:1,1:1):1,2:2);", max_proposals=8, max_samples=8)
+    assert ei.value.status == -1 and "init_newick" in str(ei.value)

@@ -176,3 +176,61 @@ def test_workspace_bytes_cfg_counts_model_buffers():
     assert f81 == P.mpcgs_workspace_bytes(12, 1000, 64, 20000, 64)
     cfg.model = P.MODELS["F84"]
     assert P.lib().mpcgs_workspace_bytes_cfg(12, 1000, ctypes.byref(cfg)) >= f81 + 64 * 11 * 32 * 8
+
+
+# ------------------------------------------------------------------ Newick G0 (SURVEY 8(b) init_newick)
+def _newick(parent, age):
+    """Plain recursive Newick writer (tips labelled by row index)."""
+    parent = np.asarray(parent)
+    nn = len(parent)
+    n = (nn + 1) // 2
+    kids = {v: [] for v in range(nn)}
+    for v in range(nn):
+        if parent[v] >= 0:
+            kids[int(parent[v])].append(v)
+    root = int(np.where(parent < 0)[0][0])
+
+    def rec(v):
+        if v < n:
+            return str(v)
+        return "(" + ",".join(f"{rec(c)}:{float(age[v] - age[c])!r}" for c in kids[v]) + ")"
+
+    return rec(root) + ";"
+
+
+def test_parse_newick_hand_example():
+    import paper_conf_ipps_davistzw17_b200 as P
+
+    # ((0,1) at 0.1, 2) at 0.4, with 3 joined at the root 1.0
+    p, a = P.mpcgs_parse_newick(4, " (((0:0.1, 1:0.1)x:0.3,2:0.4):0.6, 3:1.0);\n")
+    assert list(p) == [4, 4, 5, 6, 5, 6, -1]
+    assert np.allclose(a, [0, 0, 0, 0, 0.1, 0.4, 1.0], rtol=0, atol=1e-15)
+
+
+def test_parse_newick_roundtrip_random_trees():
+    import paper_conf_ipps_davistzw17_b200 as P
+
+    rng = np.random.default_rng(12)
+    for n in (2, 3, 5, 12, 64, 257):
+        p, a = synth.coalescent_tree(n, 0.7, rng)   # interior ids already in ascending age
+        gp, ga = P.mpcgs_parse_newick(n, _newick(p, a))
+        assert np.array_equal(gp, p)
+        assert np.allclose(ga, a, rtol=1e-13, atol=1e-15)
+
+
+@pytest.mark.parametrize("bad", [
+    "((0:0.1,1:0.1):0.3,2:0.4)",            # no ';'
+    "((0:0.1,1:0.1):0.3,2);",               # missing length
+    "((0:0.1,1:0.1):0.3,2:0.9);",           # not contemporaneous
+    "((0:0.1,1:0.1,2:0.1):0.3,3:0.4);",     # multifurcation
+    "((0:0.1,0:0.1):0.3,2:0.4);",           # duplicate tip
+    "((0:0.1,5:0.1):0.3,2:0.4);",           # label out of range
+    "((a:0.1,1:0.1):0.3,2:0.4);",           # non-numeric label
+    "((0:0.1,1:-0.1):0.3,2:0.2);",          # negative length
+    "(0:0.4,1:0.4);",                       # too few tips for n = 3
+])
+def test_parse_newick_errors(bad):
+    import paper_conf_ipps_davistzw17_b200 as P
+
+    with pytest.raises(P.MpcgsError):
+        P.mpcgs_parse_newick(3, bad)
