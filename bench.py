@@ -277,9 +277,6 @@ def main():
     world = int(os.environ.get("WORLD_SIZE", "1"))
     rank = int(os.environ.get("RANK", "0"))
     local = int(os.environ.get("LOCAL_RANK", "0"))
-    # pruning tiling policy (DESIGN 7): tile for one rank's share of the proposals at
-    # this world size (read by the library at its first launch)
-    os.environ.setdefault("MPCGS_TILING_WORLD", str(world))
     over = {}
     if args.L:
         over["L"] = args.L

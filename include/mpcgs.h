@@ -274,6 +274,13 @@ mpcgs_status mpcgs_shard_range(int32_t n_proposals, int32_t rank, int32_t world,
  * mask for an ambiguity code (S24: a site differs when the two sets are disjoint). */
 mpcgs_status mpcgs_upgma(int32_t n_seq, int32_t n_sites, const uint8_t* codes, double theta0,
                          int32_t* parent, double* age);
+/* [host-only] Site tiling of one pruning launch scoring `ntrees` genealogies (a rank's
+ * share of the proposals): tiles x sites_per_cta sites per genealogy, and the exact-sum
+ * unit in site batches.  The tiling follows ntrees; the
+ * likelihoods do not (site sums are exact over units fixed by n, L and precision, P22).
+ * Outputs nullable; MPCGS_E_ARG on n < 3, L < 1, ntrees < 1 or a bad precision. */
+mpcgs_status mpcgs_prune_tiling(int32_t n_seq, int32_t n_sites, int32_t ntrees, int32_t precision,
+                                int32_t* tiles, int32_t* sites_per_cta, int32_t* unit_batches);
 /* [host-only] Parse a Newick genealogy of n_seq tips (grammar and rules of
  * mpcgs_config.init_newick) into parent/age [2n-1] host arrays: interior ids n..2n-2 in
  * ascending age (ties: post-order), a node's age = its longest path down to a tip.

@@ -151,6 +151,150 @@ struct SiteAcc {
         if constexpr (W) return wlog;
         return mant > 0.0 ? log(mant) + (double)expo * 0.69314718055994530942 : -INFINITY;
     }
+    __device__ __forceinline__ void reset() {
+        mant = 1.0;
+        wlog = 0.0;
+        expo = 0;
+    }
 };
+
+// ---------------------------------------------------------------------------
+// Exact site sums (P22: the same logL for every tiling and world size).
+// A genealogy's ln P(D|G) (Eq. 22 read as a product, S4) is the sum of per-unit
+// terms: a unit is a fixed range of sites (a function of n, L and the precision
+// only), within which each thread multiplies its own sites' likelihoods and
+// takes one log.  Those terms are added as 128-bit two's-complement fixed point
+// with 64 fraction bits, i.e. as integers: associative, so the order in which
+// threads, CTAs and tiles add them (and hence the pruning tiling, which follows
+// the number of proposals a rank scores) cannot change the result.  Each term
+// is truncated to a multiple of 2^-64 (error < 5.5e-20 per term); the sum is
+// rounded to double once at the end.  A zero site likelihood makes the total
+// -inf (S6); |term| must stay below 2^62.
+// ---------------------------------------------------------------------------
+struct Exact128 {
+    unsigned long long lo = 0ull;
+    long long hi = 0ll;
+    unsigned flags = 0u;  // bit 0: -inf (a zero likelihood), bit 1: NaN / out of range
+
+    __device__ __forceinline__ void add_fixed(unsigned long long ql, long long qh) {
+        const unsigned long long nl = lo + ql;
+        hi += qh + (long long)(nl < lo);
+        lo = nl;
+    }
+    __device__ __forceinline__ void add(double v) {
+        if (v == 0.0) return;
+        if (!(v > -INFINITY)) {
+            flags |= (v == -INFINITY) ? 1u : 2u;
+            return;
+        }
+        const unsigned long long bits = (unsigned long long)__double_as_longlong(v);
+        int e = (int)((bits >> 52) & 0x7FFull);
+        unsigned long long m = bits & 0xFFFFFFFFFFFFFull;
+        if (e == 0x7FF) {  // +inf
+            flags |= 2u;
+            return;
+        }
+        if (e == 0) e = 1;                 // subnormal
+        else m |= 1ull << 52;
+        const int sh = e - 1075 + 64;      // |v| 2^64 = m 2^sh
+        unsigned long long ql, qh;
+        if (sh >= 74) {                    // |v| >= 2^62: outside the accumulator's range
+            flags |= 2u;
+            return;
+        } else if (sh >= 64) {
+            qh = m << (sh - 64);
+            ql = 0ull;
+        } else if (sh > 0) {
+            ql = m << sh;
+            qh = m >> (64 - sh);
+        } else if (sh > -64) {
+            ql = m >> (-sh);
+            qh = 0ull;
+        } else {
+            return;                        // below 2^-64
+        }
+        if (bits >> 63) {                  // negate (two's complement)
+            ql = ~ql + 1ull;
+            qh = ~qh + (unsigned long long)(ql == 0ull);
+        }
+        add_fixed(ql, (long long)qh);
+    }
+    __device__ __forceinline__ void add(const Exact128& o) {
+        add_fixed(o.lo, o.hi);
+        flags |= o.flags;
+    }
+    __device__ __forceinline__ void shfl_down_add(int off) {
+        Exact128 o;
+        o.lo = __shfl_down_sync(0xffffffffu, lo, off);
+        o.hi = __shfl_down_sync(0xffffffffu, hi, off);
+        o.flags = __shfl_down_sync(0xffffffffu, flags, off);
+        add(o);
+    }
+};
+
+__device__ __forceinline__ double exact_to_double(unsigned long long lo, long long hi, unsigned flags) {
+    if (flags & 2u) return __longlong_as_double(0x7FF8000000000000ll);  // NaN
+    if (flags & 1u) return -INFINITY;
+    return (double)hi + (double)lo * 5.421010862427522e-20;          // hi + lo 2^-64
+}
+
+template <int NT>
+struct ExactScratch {
+    unsigned long long w[3 * (NT / 32) + 1];
+};
+
+// Per-genealogy accumulator in device memory: [0] lo, [1] hi, [2] flags (zero on entry;
+// reset by the CTA that completes the genealogy).
+// Block-reduce v (exactly), add it to acc with 64-bit atomics (carry from the low
+// word's old value), and let the last of `tiles` CTAs write the double to *out.
+// scratch: shared memory of >= 3 * NT / 32 + 1 words, free for the call (the table
+// kernel passes its tip-code staging buffers, so the commit adds no static shared
+// memory that would cost it a fused triplet table).
+template <int NT>
+__device__ __forceinline__ void exact_commit(Exact128 v, unsigned long long* acc, unsigned* cnt, int tiles,
+                                             double* out, unsigned long long* scratch) {
+    unsigned long long* s_lo = scratch;
+    long long* s_hi = reinterpret_cast<long long*>(scratch + NT / 32);
+    unsigned long long* s_fl = scratch + 2 * (NT / 32);
+    volatile unsigned long long* s_last = scratch + 3 * (NT / 32);
+    const int tid = threadIdx.x;
+#pragma unroll
+    for (int off = 16; off > 0; off >>= 1) v.shfl_down_add(off);
+    if ((tid & 31) == 0) {
+        s_lo[tid >> 5] = v.lo;
+        s_hi[tid >> 5] = v.hi;
+        s_fl[tid >> 5] = v.flags;
+    }
+    __syncthreads();
+    if (tid == 0) {
+        Exact128 t;
+        for (int w = 0; w < NT / 32; ++w) {
+            Exact128 o;
+            o.lo = s_lo[w];
+            o.hi = s_hi[w];
+            o.flags = (unsigned)s_fl[w];
+            t.add(o);
+        }
+        const unsigned long long old = atomicAdd(acc, t.lo);
+        const unsigned long long carry = (old + t.lo < old) ? 1ull : 0ull;
+        atomicAdd(acc + 1, (unsigned long long)t.hi + carry);
+        if (t.flags) atomicOr(acc + 2, (unsigned long long)t.flags);
+        __threadfence();
+        const unsigned prev = atomicAdd(cnt, 1u);
+        *s_last = (prev == (unsigned)(tiles - 1)) ? 1ull : 0ull;
+    }
+    __syncthreads();
+    if (*s_last && tid == 0) {
+        __threadfence();
+        const volatile unsigned long long* va = acc;
+        const unsigned long long lo = va[0], hi = va[1], fl = va[2];
+        *out = exact_to_double(lo, (long long)hi, (unsigned)fl);
+        acc[0] = 0ull;
+        acc[1] = 0ull;
+        acc[2] = 0ull;
+        *cnt = 0u;
+    }
+    __syncthreads();
+}
 
 }  // namespace mpcgs

@@ -172,7 +172,7 @@ struct DevState {
     int32_t* tree_need; // [Nmax] register need of each local proposal's schedule
     uint32_t* sched_op; // [Nmax][nops]
     void* sched_e;      // [Nmax][nops] x {e_a, em_a, e_b, em_b} (float or double)
-    double* tile_part;  // [Nmax][tiles_max]
+    unsigned long long* tree_acc;  // [Nmax][4] exact site-sum accumulators (arith.cuh Exact128)
     uint32_t* tile_cnt; // [Nmax]
     // samples (5.1.3 L1264-1269: S_G suffices for Eq. 18)
     double *sS, *sL;

@@ -126,7 +126,7 @@ mpcgs_status fail(mpcgs_ctx* c, mpcgs_status st, const std::string& msg) {
 struct Layout {
     size_t codes, codes2, parent, left, right, need, age, e, em, gen, ctx_i, ctx_d, tau, len, lcnt, entry, omega, fixed;
     size_t gm, sched_P;
-    size_t tree_need, rec, sched_op, sched_e, tile_part, tile_cnt, sS, sL, sStep, sSlot, counters, last_draws, theta_buf,
+    size_t tree_need, rec, sched_op, sched_e, tree_acc, tile_cnt, sS, sL, sStep, sSlot, counters, last_draws, theta_buf,
         theta_cnt, score_out, site_w, GL, GE, path, pathsib, cpath, csib, ixyz, iee, cinfo, gen_order, total;
     int tiles_max;
 };
@@ -170,7 +170,7 @@ Layout layout(int n, int L, int Nmax, int64_t Mmax, int precision, int increment
     y.tree_need = take(4 * (size_t)Nmax);
     y.sched_op = take(4 * (size_t)Nmax * nops);
     y.sched_e = take(esz * (size_t)Nmax * nops);
-    y.tile_part = take(8 * (size_t)Nmax * y.tiles_max);
+    y.tree_acc = take(32 * (size_t)Nmax);
     y.tile_cnt = take(4 * (size_t)Nmax);
     y.sS = take(8 * (size_t)std::max<int64_t>(Mmax, 1));
     y.sL = take(8 * (size_t)std::max<int64_t>(Mmax, 1));
@@ -616,19 +616,17 @@ void upgma(int n, int L, const uint8_t* codes, double theta0, int32_t* parent, d
     }
 }
 
-// Sites per CTA: a multiple of the kernel's site batch (1..MPCGS_MAXPER = 64 batches),
-// chosen by a small cost model in units of one batch: a CTA costs its per-tree
-// setup (schedule compaction, tables: ~MPCGS_SETUP batches) plus its batches;
-// the launch takes ceil(CTAs / resident CTAs) waves of one CTA (up to four waves),
-// else total work / resident CTAs plus half a CTA of tail.  Few batches per tree and many trees -> one CTA per tree (the setup is
-// not repeated per tile); few trees -> more tiles for parallelism.  Depends only
-// on n, L, the GLOBAL tree count and the tiling policy, so every rank tiles (and
-// sums) a proposal's sites identically (world-size invariance, P22).  The policy
-// MPCGS_TILING_WORLD = P (environment, default 1) costs the waves of one rank at
-// world size P (N/P trees): a multi-GPU run sets it to its world size so that
-// each rank's share fills whole waves (results then match any other world size
-// run under the same policy bit for bit, and differ from policy 1 by FP rounding
-// of the site sums only).
+// Sites per CTA: a multiple of the kernel's exact-sum unit (unit_batches site
+// batches; 1..MPCGS_MAXPER = 64 batches), chosen by a small cost model in units of
+// one batch: a CTA costs its per-tree setup (schedule compaction, tables:
+// ~MPCGS_SETUP batches) plus its batches; the launch takes ceil(CTAs / resident
+// CTAs) waves of one CTA (up to four waves), else total work / resident CTAs plus
+// half a CTA of tail.  Few batches per tree and many trees -> one CTA per tree (the
+// setup is not repeated per tile); few trees -> more tiles for parallelism.  The
+// tree count is the number THIS launch scores (a rank's share of the proposals):
+// the site sums are exact (arith.cuh Exact128) over units fixed by the alignment,
+// so the tiling never changes a likelihood and every world size gives the same
+// chain (P22).
 #ifndef MPCGS_MAXPER
 #define MPCGS_MAXPER 64
 #endif
@@ -638,41 +636,36 @@ void upgma(int n, int L, const uint8_t* codes, double theta0, int32_t* parent, d
 #ifndef MPCGS_SETUP
 #define MPCGS_SETUP 3.0
 #endif
-static int tiling_world() {
-    static const int w = [] {
-        const char* e = std::getenv("MPCGS_TILING_WORLD");
-        const int v = e ? std::atoi(e) : 1;
-        return v >= 1 ? v : 1;
-    }();
-    return w;
-}
-
-void prune_tiling(int n, int L, int ntrees_global, int precision, int& tiles, int& sites_per_cta) {
+void prune_tiling(int n, int L, int ntrees, int precision, int& tiles, int& sites_per_cta) {
     const int batch = prune_batch_sites(n, precision);
-    const double trees = (double)ntrees_global / (double)tiling_world();  // one rank's share under the policy
+    const int unit = prune_unit_batches(n, L, precision);
+    const double trees = (double)std::max(ntrees, 1);
     const long batches = (L + batch - 1) / batch;
+    const long units = (batches + unit - 1) / unit;
     const double slots = 148.0 * (precision == 32 ? 4.0 : 3.0);  // resident CTAs (occupancy of the table kernel)
+    const long tmin = std::max<long>(1, (units * unit + MPCGS_MAXPER - 1) / MPCGS_MAXPER);
     double best = 1e300;
-    int bp = 1;
-    for (int per = 1; per <= MPCGS_MAXPER; ++per) {
-        const long t = (batches + per - 1) / per;
-        const double len = MPCGS_SETUP + (double)std::min<long>(per, batches);
+    long bt = tmin;
+    for (long t = tmin; t <= units; ++t) {
+        const long per = std::min<long>(((units + t - 1) / t) * unit, batches);  // batches of the largest tile
+        const double len = MPCGS_SETUP + (double)per;
         const double ctas = trees * (double)t;
         const double work = trees * ((double)t * MPCGS_SETUP + (double)batches);
         // a few waves: equal CTAs run in lock-step waves; many: the tail averages out
         const double cost = ctas <= 4.0 * slots ? std::ceil(ctas / slots) * len : work / slots + 0.5 * len;
         if (cost < best * (1.0 - 1e-9)) {
             best = cost;
-            bp = per;
+            bt = t;
         }
-        if (per >= batches) break;
     }
-    sites_per_cta = bp * batch;
-    tiles = (L + sites_per_cta - 1) / sites_per_cta;
+    tiles = (int)bt;
+    sites_per_cta = (int)std::min<long>(((units + bt - 1) / bt) * unit * (long)batch, (long)L);
 }
 
 // incremental rescoring (no per-CTA table setup): as many batches per CTA as
-// keep >= ~8 CTAs per SM busy, up to MPCGS_MAXPER_INCR; global N (world-size invariance)
+// keep >= ~8 CTAs per SM busy, up to MPCGS_MAXPER_INCR.  Each thread multiplies its
+// sites over the whole tile before its log, so this tiling depends on the GLOBAL
+// proposal count only (identical on every rank: P22); the tile sums are exact.
 void incr_tiling(int n, int L, int ntrees_global, int precision, int& tiles, int& sites_per_cta) {
     const int batch = prune_batch_sites(n, precision);
     const long batches = (L + batch - 1) / batch;
@@ -682,7 +675,7 @@ void incr_tiling(int n, int L, int ntrees_global, int precision, int& tiles, int
     tiles = (L + sites_per_cta - 1) / sites_per_cta;
 }
 
-PruneArgs prune_args(mpcgs_ctx* c, int ntrees_global, double* out, int out_first, int out_stride) {
+PruneArgs prune_args(mpcgs_ctx* c, int ntrees, double* out, int out_first, int out_stride) {
     PruneArgs a{};
     a.codes = c->s.codes;
     a.codes2 = c->codes2;
@@ -697,9 +690,12 @@ PruneArgs prune_args(mpcgs_ctx* c, int ntrees_global, double* out, int out_first
     a.gm = c->model ? c->s.gm : nullptr;
     a.amb = c->s.amb;
     a.sched_P = c->s.sched_P;
-    prune_tiling(c->n, c->L, ntrees_global, c->precision, a.tiles, a.sites_per_cta);
+    prune_tiling(c->n, c->L, ntrees, c->precision, a.tiles, a.sites_per_cta);
+    a.unit_batches = prune_unit_batches(c->n, c->L, c->precision);
+    a.unit_sites = a.unit_batches * prune_batch_sites(c->n, c->precision);
+    a.units = (c->L + a.unit_sites - 1) / a.unit_sites;
     a.tree_need = c->s.tree_need;
-    a.tile_part = c->s.tile_part;
+    a.tree_acc = c->s.tree_acc;
     a.tile_cnt = c->s.tile_cnt;
     a.out = out;
     a.out_first = out_first;
@@ -810,14 +806,14 @@ mpcgs_status step_local_launch(mpcgs_ctx* c, uint64_t seed, int64_t step, int N,
     int first = 1 + c->rank * (N / c->world), count = N / c->world;
     if (with_context) CU(launch_context(c->s, seed, step, c->work));
     CU(launch_propose(c->s, seed, step, first, count, c->work));
-    PruneArgs a = prune_args(c, N, c->s.rec, first, REC);
+    PruneArgs a = prune_args(c, count, c->s.rec, first, REC);
     if (pre) CU(cudaEventRecord(pre, c->work));
     int np = 1;
     if (c->incremental) {
         IncrArgs ia{};
         ia.count = count;
         incr_tiling(c->n, c->L, N, c->precision, ia.tiles, ia.sites_per_cta);
-        ia.tile_part = c->s.tile_part;
+        ia.tree_acc = c->s.tree_acc;
         ia.tile_cnt = c->s.tile_cnt;
         ia.out = c->s.rec;
         ia.out_first = first;
@@ -928,6 +924,17 @@ int32_t mpcgs_tree_schedule(int32_t n, const int32_t* parent, const double* age,
     HostTree ht;
     host_tree(n, parent, age, mu, ht);
     return host_schedule<double>(n, ht, op, e);
+}
+
+mpcgs_status mpcgs_prune_tiling(int32_t n, int32_t L, int32_t ntrees, int32_t precision, int32_t* tiles,
+                                int32_t* sites_per_cta, int32_t* unit_batches) {
+    if (n < 3 || n > MPCGS_MAX_SEQ || L < 1 || ntrees < 1 || (precision != 32 && precision != 64)) return MPCGS_E_ARG;
+    int t = 0, spc = 0;
+    prune_tiling(n, L, ntrees, precision, t, spc);
+    if (tiles) *tiles = t;
+    if (sites_per_cta) *sites_per_cta = spc;
+    if (unit_batches) *unit_batches = prune_unit_batches(n, L, precision);
+    return MPCGS_OK;
 }
 
 mpcgs_status mpcgs_parse_newick(int32_t n, const char* newick, int32_t* parent, double* age) {
@@ -1236,7 +1243,7 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
         s.tree_need = (int32_t*)(b + y.tree_need);
         s.sched_op = (uint32_t*)(b + y.sched_op);
         s.sched_e = (void*)(b + y.sched_e);
-        s.tile_part = (double*)(b + y.tile_part);
+        s.tree_acc = (unsigned long long*)(b + y.tree_acc);
         s.tile_cnt = (uint32_t*)(b + y.tile_cnt);
         s.sS = (double*)(b + y.sS);
         s.sL = (double*)(b + y.sL);

@@ -124,8 +124,6 @@ __global__ void __launch_bounds__(INCR_THREADS) k_score_incr(DevState s, IncrArg
     __shared__ double sh_pe[4 * 128];   // e, em of the path branches and of the siblings' branches
     __shared__ int sh_xyz[INCR_PG][4];
     __shared__ double sh_ee[INCR_PG][10];
-    __shared__ double s_red[INCR_THREADS / 32];
-    __shared__ bool s_last;
     using T2 = typename std::conditional<sizeof(T) == 8, double2, float2>::type;
     __shared__ __align__(16) T2 sB[INCR_DC][2][INCR_THREADS];  // B_a of this thread's current site (conflict-free halves)
     __shared__ int sBE[INCR_DC][INCR_THREADS];
@@ -240,34 +238,16 @@ __global__ void __launch_bounds__(INCR_THREADS) k_score_incr(DevState s, IncrArg
             }
         }
     }
+    // per proposal: this thread's log over the tile, summed exactly (arith.cuh Exact128)
+    __shared__ ExactScratch<INCR_THREADS> s_ex;
 #pragma unroll
     for (int j = 0; j < INCR_PG; ++j) {
-        if (j >= np) break;
-        double ll = acc[j].total();
-#pragma unroll
-        for (int off = 16; off > 0; off >>= 1) ll += __shfl_down_sync(0xffffffffu, ll, off);
-        if ((tid & 31) == 0) s_red[tid >> 5] = ll;
-        __syncthreads();
-        if (tid == 0) {
-            double t = 0.0;
-            for (int w = 0; w < INCR_THREADS / 32; ++w) t += s_red[w];
-            const int tree = p0 + j;
-            a.tile_part[(size_t)tree * a.tiles + tile] = t;
-            __threadfence();
-            const unsigned prev = atomicAdd(a.tile_cnt + tree, 1u);
-            s_last = (prev == (unsigned)(a.tiles - 1));
-        }
-        __syncthreads();
-        if (s_last && tid == 0) {
-            __threadfence();
-            const int tree = p0 + j;
-            double t = 0.0;
-            const volatile double* tp = a.tile_part + (size_t)tree * a.tiles;
-            for (int k = 0; k < a.tiles; ++k) t += tp[k];
-            a.out[(size_t)(a.out_first + tree) * a.out_stride] = t;
-            a.tile_cnt[tree] = 0u;
-        }
-        __syncthreads();
+        if (j >= np) break;  // np is uniform in the CTA
+        Exact128 ex;
+        ex.add(acc[j].total());
+        const int tree = p0 + j;
+        exact_commit<INCR_THREADS>(ex, a.tree_acc + 4 * (size_t)tree, a.tile_cnt + tree, a.tiles,
+                                   a.out + (size_t)(a.out_first + tree) * a.out_stride, s_ex.w);
     }
 }
 

@@ -31,16 +31,30 @@ struct PruneArgs {
     const double* gm;          // general model (f4): [36] eigen-system of Q, else nullptr (F81)
     void* sched_P;             // general model: [ntrees][nops][32] P matrices (float / double)
     int amb;                   // byte codes are base-set masks (ambiguity codes): flat kernel only
-    int tiles, sites_per_cta;
+    // site tiles: tile t covers exact-sum units [t*units/tiles, (t+1)*units/tiles) of
+    // unit_sites sites each (balanced; tile_range below); sites_per_cta = the largest tile
+    int tiles, sites_per_cta, units, unit_sites;
     const double* site_w;      // [L] pattern counts (compressed sites, f3) or nullptr
     const int32_t* tree_need;  // [ntrees] register need of each tree's schedule (nullable)
     int need_cap;              // set by launch_prune: largest need the table kernel serves
     int trip_cap;              // set by launch_prune: fused triplets per tree (table kernel)
-    double* tile_part;         // [ntrees][tiles]
+    int unit_batches;          // table kernel: site batches per exact-sum unit (tiles hold whole units)
+    unsigned long long* tree_acc;  // [ntrees][4] exact site-sum accumulators (Exact128), zero on entry
     uint32_t* tile_cnt;        // [ntrees], zero on entry, reset by the kernel
     double* out;               // logL of tree t -> out[(out_first + t) * out_stride]
     int out_first, out_stride;
 };
+__device__ __forceinline__ void tile_range(const PruneArgs& a, int tile, int& s_begin, int& s_end) {
+    const int u0 = (int)(((long long)tile * a.units) / a.tiles);
+    const int u1 = (int)(((long long)(tile + 1) * a.units) / a.tiles);
+    s_begin = u0 * a.unit_sites;
+    s_end = min(a.L, u1 * a.unit_sites);
+}
+constexpr int FLAT_UNIT_SITES = 256;  // flat kernel: sites per exact-sum unit (tiles hold whole units)
+// site batches per exact-sum unit of the table kernel: a function of the alignment
+// only (never of the number of proposals or ranks), so that every tiling a rank may
+// choose sums the same terms (P22)
+int prune_unit_batches(int n, int L, int precision);
 
 int prune_depth_for(int n);
 int prune_max_need(int n);
@@ -64,7 +78,7 @@ cudaError_t launch_fill_gen_record(const DevState& s, cudaStream_t st);
 struct IncrArgs {
     int count;                 // proposals of this rank (local slots 0..count-1)
     int tiles, sites_per_cta;
-    double* tile_part;         // [count][tiles]
+    unsigned long long* tree_acc;  // [count][4] exact site-sum accumulators
     uint32_t* tile_cnt;        // [count]
     double* out;               // logL of local proposal t -> out[(out_first + t) * out_stride]
     int out_first, out_stride;

@@ -28,6 +28,18 @@ static int prune_si(int n, int precision) {
 }
 int prune_batch_sites(int n, int precision) { return PRUNE_THREADS * prune_si(n, precision); }
 
+// exact-sum units (arith.cuh Exact128): one log per thread per unit; 4-batch units on
+// long alignments (the tiling is coarse there anyway), single batches below
+// MPCGS_UNIT_MIN_BATCHES batches.  A function of the alignment only (P22).
+#ifndef MPCGS_UNIT_MIN_BATCHES
+#define MPCGS_UNIT_MIN_BATCHES 32
+#endif
+int prune_unit_batches(int n, int L, int precision) {
+    const int batch = prune_batch_sites(n, precision);
+    const long batches = (L + batch - 1) / batch;
+    return batches >= MPCGS_UNIT_MIN_BATCHES ? 4 : 1;
+}
+
 // register need the table kernel serves (DR registers + PRUNE_SPILL shared levels);
 // deeper trees (rare) are scored by the flat kernel in a second pass
 // One shared spill level up to n = 64 (a random coalescent tree of 64 tips needs

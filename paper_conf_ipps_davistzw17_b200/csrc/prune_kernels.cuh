@@ -187,8 +187,6 @@ __global__ void __launch_bounds__(PRUNE_THREADS) k_prune(PruneArgs a) {
     extern __shared__ __align__(16) unsigned char smem_raw[];
     E4* s_e = reinterpret_cast<E4*>(smem_raw);
     uint32_t* s_op = reinterpret_cast<uint32_t*>(smem_raw + sizeof(E4) * a.nops);
-    __shared__ double s_red[PRUNE_THREADS / 32];
-    __shared__ bool s_last;
 
     const int tree = blockIdx.y;
     const int tile = blockIdx.x;
@@ -205,71 +203,57 @@ __global__ void __launch_bounds__(PRUNE_THREADS) k_prune(PruneArgs a) {
     const T pi[4] = {(T)a.pi[0], (T)a.pi[1], (T)a.pi[2], (T)a.pi[3]};
     const uint8_t* __restrict__ codes = a.codes;
     const int Lpad = a.Lpad;
-    const int s_begin = tile * a.sites_per_cta;
-    const int s_end = min(a.L, s_begin + a.sites_per_cta);
+    int s_begin, s_end;
+    tile_range(a, tile, s_begin, s_end);
 
     SiteAcc<W> acc;
+    Exact128 ex;
     T R[D][4];
 #pragma unroll
     for (int i = 0; i < D; ++i)
 #pragma unroll
         for (int j = 0; j < 4; ++j) R[i][j] = T(0);
 
-    for (int site = s_begin + threadIdx.x; site < s_end; site += blockDim.x) {
-        int scale = 0;
-        for (int op = 0; op < a.nops; ++op) {
-            const uint32_t code = s_op[op];
-            if constexpr (GM) {
-                const T* __restrict__ P = gP + (size_t)op * 32;
-                switch (code & 63u) {
-                    MPCGS_GMCASE(0) MPCGS_GMCASE(1) MPCGS_GMCASE(2) MPCGS_GMCASE(3) MPCGS_GMCASE(4)
-                    MPCGS_GMCASE(5) MPCGS_GMCASE(6) MPCGS_GMCASE(7) MPCGS_GMCASE(8) MPCGS_GMCASE(9)
-                    MPCGS_GMCASE(10) MPCGS_GMCASE(11)
-                    default: break;
-                }
-            } else {
-                const E4 ed = s_e[op];
-                switch (code & 63u) {
-                    MPCGS_OPCASE(0) MPCGS_OPCASE(1) MPCGS_OPCASE(2) MPCGS_OPCASE(3) MPCGS_OPCASE(4)
-                    MPCGS_OPCASE(5) MPCGS_OPCASE(6) MPCGS_OPCASE(7) MPCGS_OPCASE(8) MPCGS_OPCASE(9)
-                    MPCGS_OPCASE(10) MPCGS_OPCASE(11)
-                    default: break;
+    // exact-sum units of FLAT_UNIT_SITES sites (tiles hold whole units, P22)
+    for (int u0 = s_begin; u0 < s_end; u0 += FLAT_UNIT_SITES) {
+        const int u1 = min(s_end, u0 + FLAT_UNIT_SITES);
+        for (int site = u0 + threadIdx.x; site < u1; site += blockDim.x) {
+            int scale = 0;
+            for (int op = 0; op < a.nops; ++op) {
+                const uint32_t code = s_op[op];
+                if constexpr (GM) {
+                    const T* __restrict__ P = gP + (size_t)op * 32;
+                    switch (code & 63u) {
+                        MPCGS_GMCASE(0) MPCGS_GMCASE(1) MPCGS_GMCASE(2) MPCGS_GMCASE(3) MPCGS_GMCASE(4)
+                        MPCGS_GMCASE(5) MPCGS_GMCASE(6) MPCGS_GMCASE(7) MPCGS_GMCASE(8) MPCGS_GMCASE(9)
+                        MPCGS_GMCASE(10) MPCGS_GMCASE(11)
+                        default: break;
+                    }
+                } else {
+                    const E4 ed = s_e[op];
+                    switch (code & 63u) {
+                        MPCGS_OPCASE(0) MPCGS_OPCASE(1) MPCGS_OPCASE(2) MPCGS_OPCASE(3) MPCGS_OPCASE(4)
+                        MPCGS_OPCASE(5) MPCGS_OPCASE(6) MPCGS_OPCASE(7) MPCGS_OPCASE(8) MPCGS_OPCASE(9)
+                        MPCGS_OPCASE(10) MPCGS_OPCASE(11)
+                        default: break;
+                    }
                 }
             }
+            // Eq. 21: L_s = sum_X pi_X L_root(X), root partial in R[0]
+            T ls = pi[0] * R[0][0];
+            ls = fma(pi[1], R[0][1], ls);
+            ls = fma(pi[2], R[0][2], ls);
+            ls = fma(pi[3], R[0][3], ls);
+            acc.add((double)ls, scale, a.site_w, site);
         }
-        // Eq. 21: L_s = sum_X pi_X L_root(X), root partial in R[0]
-        T ls = pi[0] * R[0][0];
-        ls = fma(pi[1], R[0][1], ls);
-        ls = fma(pi[2], R[0][2], ls);
-        ls = fma(pi[3], R[0][3], ls);
-        acc.add((double)ls, scale, a.site_w, site);
+        // ln of this thread's product over the unit (0 if it had no site); -inf if a
+        // site likelihood was 0 (S6)
+        ex.add(acc.total());
+        acc.reset();
     }
-    // ln of this thread's product; -inf if any site likelihood was 0 (S6)
-    double ll = acc.total();
-    if (s_begin + (int)threadIdx.x >= s_end) ll = 0.0;
-
-    // block reduction in a fixed order
-#pragma unroll
-    for (int off = 16; off > 0; off >>= 1) ll += __shfl_down_sync(0xffffffffu, ll, off);
-    if ((threadIdx.x & 31) == 0) s_red[threadIdx.x >> 5] = ll;
-    __syncthreads();
-    if (threadIdx.x == 0) {
-        double t = 0.0;
-        for (int w = 0; w < (int)(blockDim.x >> 5); ++w) t += s_red[w];
-        a.tile_part[(size_t)tree * a.tiles + tile] = t;
-        __threadfence();
-        unsigned prev = atomicAdd(a.tile_cnt + tree, 1u);
-        s_last = (prev == (unsigned)(a.tiles - 1));
-    }
-    __syncthreads();
-    if (s_last && threadIdx.x == 0) {
-        __threadfence();
-        double t = 0.0;
-        const volatile double* tp = a.tile_part + (size_t)tree * a.tiles;
-        for (int k = 0; k < a.tiles; ++k) t += tp[k];
-        a.out[(size_t)(a.out_first + tree) * a.out_stride] = t;
-        a.tile_cnt[tree] = 0u;
-    }
+    __shared__ ExactScratch<PRUNE_THREADS> s_ex;
+    exact_commit<PRUNE_THREADS>(ex, a.tree_acc + 4 * (size_t)tree, a.tile_cnt + tree, a.tiles,
+                                a.out + (size_t)(a.out_first + tree) * a.out_stride, s_ex.w);
 }
 
 // ============================================================================
@@ -779,15 +763,13 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
     int* s_d = reinterpret_cast<int*>(reinterpret_cast<unsigned char*>(s_spill) +
                                       sizeof(T) * (size_t)spill_lv * SI * 4 * PRUNE_THREADS);
     int* s_tl = s_d + align16(sizeof(int) * 2 * (size_t)nops) / sizeof(int);  // original codes, then check flags
-    __shared__ double s_red[PRUNE_THREADS / 32];
-    __shared__ bool s_last;
     __shared__ int s_nc;  // compacted op count
 
     const int tid = threadIdx.x;
     const int tree = blockIdx.y;
     const int tile = blockIdx.x;
-    const int s_begin = tile * a.sites_per_cta;
-    const int s_end = min(a.L, s_begin + a.sites_per_cta);
+    int s_begin, s_end;
+    tile_range(a, tile, s_begin, s_end);
     const int nb = (s_end - s_begin + BATCH - 1) / BATCH;
     if (a.tree_need && a.tree_need[tree] > a.need_cap) return;  // deeper tree: scored by the flat pass
 
@@ -1082,6 +1064,7 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
     }
 
     SiteAcc<W> acc;
+    Exact128 ex;
     Stack<T, DR, SI> st;
     st.sm = smem_addr(s_spill + tid);
 #pragma unroll
@@ -1094,64 +1077,53 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
     CD cc;
     cc.init(tid);
     const uint32_t s_tab_a = smem_addr(s_tab), s_opc_a = smem_addr(s_opc);
-    for (int b = 0; b < nb; ++b) {
-        if (b + 1 < nb) {
-            issue(b + 1, (b + 1) & 1);
-            cp_async_wait<1>();
-        } else {
-            cp_async_wait<0>();
-        }
-        __syncthreads();
-        cc.sbase = smem_addr(s_cod + (size_t)(b & 1) * bufb);
-        int scale[SI];
+    // exact-sum units of unit_batches batches (the tile starts on a unit boundary); the
+    // unit loop keeps the flush out of the batch loop
+    for (int b0 = 0; b0 < nb; b0 += a.unit_batches) {
+        const int b1 = min(nb, b0 + a.unit_batches);
+        for (int b = b0; b < b1; ++b) {
+            if (b + 1 < nb) {
+                issue(b + 1, (b + 1) & 1);
+                cp_async_wait<1>();
+            } else {
+                cp_async_wait<0>();
+            }
+            __syncthreads();
+            cc.sbase = smem_addr(s_cod + (size_t)(b & 1) * bufb);
+            int scale[SI];
 #pragma unroll
-        for (int k = 0; k < SI; ++k) scale[k] = 0;
-        for (int op = 0; op < nops_run; ++op) {
-            const uint32_t oa = s_opc_a + (uint32_t)op * (uint32_t)sizeof(OpRec<T>);
-            const uint4 ox = lds_u4(oa);
-            T up[2];
-            lds2(up, oa + 16u);
-            const UpBr<T, GM> ub(up, s_P);
-            const int di = (int)((ox.x >> 2) & 15u) * 4 + (int)(ox.x & 3u);  // dense (sp, type) index
-            run_op<T, DR, SI, PT, DMX, GM>(di, st, ox.x, ox.y, ox.w, cc.word((ox.x >> 6) & 2047), ub, s_tab_a, cc,
-                                           pi, scale);
-        }
-        const int site0 = s_begin + b * BATCH + tid * SI;
+            for (int k = 0; k < SI; ++k) scale[k] = 0;
+            for (int op = 0; op < nops_run; ++op) {
+                const uint32_t oa = s_opc_a + (uint32_t)op * (uint32_t)sizeof(OpRec<T>);
+                const uint4 ox = lds_u4(oa);
+                T up[2];
+                lds2(up, oa + 16u);
+                const UpBr<T, GM> ub(up, s_P);
+                const int di = (int)((ox.x >> 2) & 15u) * 4 + (int)(ox.x & 3u);  // dense (sp, type) index
+                run_op<T, DR, SI, PT, DMX, GM>(di, st, ox.x, ox.y, ox.w, cc.word((ox.x >> 6) & 2047), ub, s_tab_a,
+                                               cc, pi, scale);
+            }
+            const int site0 = s_begin + b * BATCH + tid * SI;
 #pragma unroll
-        for (int k = 0; k < SI; ++k) {
-            T root[4];
-            st.template get<0>(k, root);
-            T ls = pi[0] * root[0];   // Eq. 21
-            ls = fma(pi[1], root[1], ls);
-            ls = fma(pi[2], root[2], ls);
-            ls = fma(pi[3], root[3], ls);
-            if (site0 + k < s_end) acc.add((double)ls, scale[k], a.site_w, site0 + k);  // padding not counted
+            for (int k = 0; k < SI; ++k) {
+                T root[4];
+                st.template get<0>(k, root);
+                T ls = pi[0] * root[0];   // Eq. 21
+                ls = fma(pi[1], root[1], ls);
+                ls = fma(pi[2], root[2], ls);
+                ls = fma(pi[3], root[3], ls);
+                if (site0 + k < s_end) acc.add((double)ls, scale[k], a.site_w, site0 + k);  // padding not counted
+            }
+            __syncthreads();  // the buffer of batch b is refilled in iteration b+1
         }
-        __syncthreads();  // the buffer of batch b is refilled in iteration b+1
+        // this thread's log over the unit (0 if it had no site there)
+        ex.add(acc.total());
+        acc.reset();
     }
-    double ll = acc.total();
-
-#pragma unroll
-    for (int off = 16; off > 0; off >>= 1) ll += __shfl_down_sync(0xffffffffu, ll, off);
-    if ((tid & 31) == 0) s_red[tid >> 5] = ll;
-    __syncthreads();
-    if (tid == 0) {
-        double t = 0.0;
-        for (int w = 0; w < PRUNE_THREADS / 32; ++w) t += s_red[w];
-        a.tile_part[(size_t)tree * a.tiles + tile] = t;
-        __threadfence();
-        const unsigned prev = atomicAdd(a.tile_cnt + tree, 1u);
-        s_last = (prev == (unsigned)(a.tiles - 1));
-    }
-    __syncthreads();
-    if (s_last && tid == 0) {
-        __threadfence();
-        double t = 0.0;
-        const volatile double* tp = a.tile_part + (size_t)tree * a.tiles;
-        for (int k = 0; k < a.tiles; ++k) t += tp[k];
-        a.out[(size_t)(a.out_first + tree) * a.out_stride] = t;
-        a.tile_cnt[tree] = 0u;
-    }
+    // the code staging buffers are free now (the last batch ended with a barrier)
+    exact_commit<PRUNE_THREADS>(ex, a.tree_acc + 4 * (size_t)tree, a.tile_cnt + tree, a.tiles,
+                                a.out + (size_t)(a.out_first + tree) * a.out_stride,
+                                reinterpret_cast<unsigned long long*>(s_cod));
 }
 
 template <typename T, int D, bool W, bool GM, bool AMB>

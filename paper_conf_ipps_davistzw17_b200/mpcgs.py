@@ -89,6 +89,7 @@ _SIGS = {
     "mpcgs_upgma": (_i32, [_i32, _i32, _P, _f64, _P, _P]),
     "mpcgs_tree_schedule": (_i32, [_i32, _P, _P, _f64, _P, _P]),
     "mpcgs_parse_newick": (_i32, [_i32, ctypes.c_char_p, _P, _P]),
+    "mpcgs_prune_tiling": (_i32, [_i32, _i32, _i32, _i32, _P, _P, _P]),
     "mpcgs_phylip_dims": (_i32, [ctypes.c_char_p, _P, _P]),
     "mpcgs_phylip_read": (_i32, [ctypes.c_char_p, _P, _i32]),
     "mpcgs_philox": (None, [_P, _P, _P]),
@@ -109,6 +110,8 @@ def lib(build_if_missing: bool = True):
             raise MpcgsError(-4, f"CUDA library missing: {path}")
         L = ctypes.CDLL(path)
         for name, (res, args) in _SIGS.items():
+            if path != _build.LIB and not hasattr(L, name):
+                continue  # an older tuning variant (A/B runs) may lack newer entry points
             f = getattr(L, name)
             f.restype = res
             f.argtypes = args
@@ -172,6 +175,15 @@ def mpcgs_tree_schedule(parent, age, mu):
     if d < 0:
         raise MpcgsError(d, "tree_schedule")
     return op, e.reshape(n - 1, 4), d
+
+
+def mpcgs_prune_tiling(n_seq, n_sites, ntrees, precision=64):
+    """(tiles, sites_per_cta, unit_batches) of one pruning launch over ntrees genealogies."""
+    t, s, u = ctypes.c_int32(), ctypes.c_int32(), ctypes.c_int32()
+    st = lib().mpcgs_prune_tiling(n_seq, n_sites, ntrees, precision, ctypes.byref(t), ctypes.byref(s), ctypes.byref(u))
+    if st:
+        raise MpcgsError(st, "prune_tiling")
+    return t.value, s.value, u.value
 
 
 def mpcgs_parse_newick(n_seq, newick):

@@ -1,6 +1,6 @@
 """Aggregate ncu warp-stall samples of one kernel by CUDA source line.
 usage: python tools_linesamples.py REPORT.ncu-rep CUBIN MANGLED_NAME [top]"""
-import csv, re, subprocess, sys
+import csv, os, re, subprocess, sys
 from collections import defaultdict
 rep, cubin, fn = sys.argv[1:4]
 top = int(sys.argv[4]) if len(sys.argv) > 4 else 30
@@ -29,7 +29,7 @@ tot = sum(agg.values())
 src = {}
 for (f, l) in agg:
     try:
-        src[(f, l)] = open(f"paper_conf_ipps_davistzw17_b200/csrc/{f}").read().splitlines()[l - 1].strip()[:70]
+        src[(f, l)] = open(os.environ.get("SRCDIR", "paper_conf_ipps_davistzw17_b200/csrc") + f"/{f}").read().splitlines()[l - 1].strip()[:70]
     except Exception:
         src[(f, l)] = ""
 for k, v in sorted(agg.items(), key=lambda kv: -kv[1])[:top]:
