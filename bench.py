@@ -12,11 +12,14 @@ target is stated; it fits one GPU).  Inputs are synthetic: an ms-style
 coalescent tree at theta = 1 and F81 sequences with uniform pi (synth/).
 
 Timing: W untimed warm-up steps, then K steps timed on the device with CUDA
-events on the library's stream (step boundaries and every pruning launch),
-L2 flushed (256 MiB write) between timed steps outside the timed intervals;
-barrier + synchronize on both sides; max over ranks.  nvidia-smi samples the
-clocks during the timed region.  `--impl reference` times the plain CPU oracle
-(oracle/) on a bounded sample of the same workload.
+events on the library's stream (step boundaries and every phase: context +
+proposals, pruning, exchange + draws), L2 flushed (256 MiB memset on the same
+stream) between timed steps outside the timed intervals; barrier + synchronize
+on both sides; max over ranks.  nvidia-smi samples the clocks during the timed
+region.  The roofline peak is this GPU's FMA throughput measured by a
+microbenchmark (mpcgs_probe_peak) before the timed region.  `--impl reference`
+times the plain CPU oracle (oracle/) on all host cores on a bounded sample of
+the same workload.
 """
 from __future__ import annotations
 
@@ -54,6 +57,7 @@ def flops_per_site_gm(n: int) -> int:
 
 
 def peaks():
+    """Derived FMA peaks (unit counts x clock) and the driver's MEASURED_PEAKS.json."""
     mp = {}
     try:
         mp = json.load(open(os.path.join(ROOT, "MEASURED_PEAKS.json")))
@@ -62,6 +66,38 @@ def peaks():
     mhz = float(mp.get("sm_max_mhz", 1965.0))
     # B200: 148 SMs; per SM per clock 64 FP64 FMA lanes, 128 FP32 FMA lanes (FMA = 2 flops)
     return {64: 148 * 64 * 2 * mhz * 1e6 / 1e12, 32: 148 * 128 * 2 * mhz * 1e6 / 1e12}, mhz, mp
+
+
+def measured_alu_peaks(P):
+    """Microbenchmarked FP64 / FP32 FMA throughput (TFLOP/s) and shared-memory load
+    bandwidth (GB/s) of this GPU (mpcgs_probe_peak, csrc/probe.cu), measured before
+    the timed region."""
+    return {64: P.mpcgs_probe_peak(0), 32: P.mpcgs_probe_peak(1), "lds_gbs": P.mpcgs_probe_peak(2)}
+
+
+def pipe_from_profiles(tag: str):
+    """ncu pipe utilisation of the dominant kernel (profiles/prune_pipe.json, written by
+    tools/ncu_pipe_json.py from a --set full capture of the same command)."""
+    try:
+        return json.load(open(os.path.join(ROOT, "profiles", "prune_pipe.json"))).get(tag)
+    except Exception:
+        return None
+
+
+def cpu_info():
+    model = None
+    try:
+        out = subprocess.run(["lscpu"], capture_output=True, text=True, timeout=10).stdout
+        for ln in out.splitlines():
+            if ln.startswith("Model name"):
+                model = ln.split(":", 1)[1].strip()
+    except Exception:
+        pass
+    try:
+        usable = len(os.sched_getaffinity(0))
+    except Exception:
+        usable = os.cpu_count() or 1
+    return model, usable
 
 
 class Clocks:
@@ -118,62 +154,100 @@ def oracle_gen_logL(oracle, codes, parent, age, pi, u, model, kappa):
     return oracle.log_likelihood_model(model, kappa, codes, parent, age, pi)
 
 
-def cpu_oracle_sample(wl, seconds: float, n_prop: int = 1, model="F81", kappa=0.0):
-    """Time the oracle's GMH step on the same workload (bounded: n_prop proposals)."""
+def cpu_oracle_sample(wl, seconds: float, threads: int = 1, model="F81", kappa=0.0):
+    """Time the oracle (as it stands, never tuned) on the workload: the proposals of
+    consecutive GMH steps (orc_propose, then orc_log_likelihood of each, Eq. 19-22 in
+    log space), `threads` proposals at a time on that many host threads (ctypes
+    releases the GIL), until `seconds` have passed.  Returns partials/s, proposals, s."""
+    import concurrent.futures
+
     import oracle
 
     codes = wl["codes"]
     pi = oracle.base_freqs(codes)
     u = oracle.default_rate(pi)
     parent, age = wl["true_parent"], wl["true_age"]
-    gl = oracle_gen_logL(oracle, codes, parent, age, pi, u, model, kappa)
     n, L = codes.shape
-    steps, t0 = 0, time.perf_counter()
-    while True:
-        tr = oracle.gmh_step(codes, pi, u, wl["theta0"], n_prop, n_prop, wl["chain_seed"], steps, parent, age, gl,
-                             model=model, kappa=kappa)
-        parent, age, gl = tr["parent"], tr["age"], tr["gen_logL"]
-        steps += 1
-        if time.perf_counter() - t0 >= seconds:
-            break
+
+    def score(tree):
+        p2, a2 = tree
+        return oracle_gen_logL(oracle, codes, p2, a2, pi, u, model, kappa)
+
+    done, step, t0 = 0, 0, time.perf_counter()
+    with concurrent.futures.ThreadPoolExecutor(max_workers=threads) as ex:
+        while True:
+            target = oracle.pick_target(parent, wl["chain_seed"], step)
+            trees = [oracle.propose(parent, age, wl["theta0"], target, wl["chain_seed"], step, 1 + k)[:2]
+                     for k in range(threads)]
+            list(ex.map(score, trees))
+            done += threads
+            step += 1
+            if time.perf_counter() - t0 >= seconds:
+                break
     dt = time.perf_counter() - t0
-    partials = steps * n_prop * L * (n - 1)
-    return partials / dt, steps, dt
+    return done * L * (n - 1) / dt, done, dt
+
+
+def cpu_baselines(wl, seconds, model, kappa):
+    """1-thread and all-core oracle rates: the all-core leg scores one
+    proposal per host thread."""
+    cpu_model, usable = cpu_info()
+    v1, k1, t1 = cpu_oracle_sample(wl, seconds / 2, 1, model, kappa)
+    vn, kn, tn = cpu_oracle_sample(wl, seconds / 2, usable, model, kappa)
+    n, L = wl["codes"].shape
+    return {"value": vn, "unit": UNIT, "cores": usable, "kind": "oracle", "cpu_model": cpu_model,
+            "sample": f"{kn} proposals of consecutive GMH steps, each scored over all {L} sites by the oracle, "
+                      f"{usable} at a time on {usable} threads ({tn:.1f} s)",
+            "single_thread": {"value": v1, "cores": 1,
+                              "sample": f"{k1} proposals scored one after another ({t1:.1f} s)"}}
 
 
 def run_reference(args, wl, rank):
+    """The oracle as it stands (oracle/), timed on the host cores: each step scores one
+    proposal per usable host thread (the proposals of consecutive GMH steps); W warm-up
+    steps, then K steps.  Rank 0 only."""
     if rank != 0:
         return
-    codes = wl["codes"]
-    n, L = codes.shape
+    import concurrent.futures
+
     import oracle
 
+    codes = wl["codes"]
+    n, L = codes.shape
     pi = oracle.base_freqs(codes)
     u = oracle.default_rate(pi)
     parent, age = wl["true_parent"], wl["true_age"]
-    gl = oracle_gen_logL(oracle, codes, parent, age, pi, u, args.model, args.kappa)
-    n_prop = 1
-    mk = dict(model=args.model, kappa=args.kappa)
-    for s in range(args.warmup):
-        tr = oracle.gmh_step(codes, pi, u, wl["theta0"], n_prop, n_prop, wl["chain_seed"], s, parent, age, gl, **mk)
-        parent, age, gl = tr["parent"], tr["age"], tr["gen_logL"]
-    t0 = time.perf_counter()
-    for s in range(args.steps):
-        tr = oracle.gmh_step(codes, pi, u, wl["theta0"], n_prop, n_prop, wl["chain_seed"], args.warmup + s,
-                             parent, age, gl, **mk)
-        parent, age, gl = tr["parent"], tr["age"], tr["gen_logL"]
-    dt = time.perf_counter() - t0
-    partials = args.steps * n_prop * L * (n - 1)
+    cpu_model, threads = cpu_info()
+
+    def score(tree):
+        return oracle_gen_logL(oracle, codes, tree[0], tree[1], pi, u, args.model, args.kappa)
+
+    def step(s, ex):
+        target = oracle.pick_target(parent, wl["chain_seed"], s)
+        trees = [oracle.propose(parent, age, wl["theta0"], target, wl["chain_seed"], s, 1 + k)[:2]
+                 for k in range(threads)]
+        list(ex.map(score, trees))
+
+    with concurrent.futures.ThreadPoolExecutor(max_workers=threads) as ex:
+        for s in range(args.warmup):
+            step(s, ex)
+        t0 = time.perf_counter()
+        for s in range(args.steps):
+            step(args.warmup + s, ex)
+        dt = time.perf_counter() - t0
+    partials = args.steps * threads * L * (n - 1)
     value = partials / dt
-    sample = f"oracle GMH step with {n_prop} proposal (of {wl['N']}) over all {L} sites, {args.steps} steps"
+    sample = (f"per step {threads} proposals (of {wl['N']}) resimulated and scored over all {L} sites by the "
+              f"oracle, one per host thread, {args.steps} steps")
     line = {
         "impl": "reference", "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": args.gpus,
         "steps": args.steps, "warmup": args.warmup, "ms_per_step": 1e3 * dt / args.steps,
         "higher_is_better": True, "scaling": "strong", "vs_baseline": None, "dtype": "f64", "data": "synthetic",
         "config": workload_config(args, wl),
-        "cpu_baseline": {"value": value, "unit": UNIT, "cores": 1, "kind": "oracle", "sample": sample},
+        "cpu_baseline": {"value": value, "unit": UNIT, "cores": threads, "kind": "oracle", "sample": sample,
+                         "cpu_model": cpu_model},
         "e2e": {"value": value, "unit": UNIT, "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
-        "proposals_per_s": args.steps * n_prop / dt,
+        "proposals_per_s": args.steps * threads / dt,
     }
     print(json.dumps(line), flush=True)
 
@@ -256,7 +330,8 @@ def main():
     ap.add_argument("--n", type=int, default=None)
     ap.add_argument("--N", type=int, default=None)
     ap.add_argument("--precision", type=int, default=64, choices=[32, 64])
-    ap.add_argument("--cpu-seconds", type=float, default=12.0)
+    ap.add_argument("--cpu-seconds", type=float, default=20.0,
+                    help="host time for the oracle baselines (half 1 thread, half all cores)")
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--no-incremental-block", action="store_true")
     ap.add_argument("--compress", action="store_true",
@@ -335,6 +410,7 @@ def main():
                     init_tree=(wl["true_parent"], wl["true_age"]), rank=rank, world=world, nccl_id=nccl_id,
                     stream=stream, incremental=args.incremental, compress_patterns=args.compress,
                     model=args.model, kappa=args.kappa, ambiguity=args.ambiguity > 0)
+    alu = measured_alu_peaks(P)  # FMA / shared-memory microbenchmarks, before the timed region
     # warm-up (untimed): W steps
     ctx.mpcgs_sample(N, N * args.warmup, wl["chain_seed"])
     ctx.mpcgs_set_timing(3)   # per-step + per-prune CUDA events, L2 flush between steps
@@ -343,11 +419,12 @@ def main():
     ctx.mpcgs_sample(N, N * args.steps, wl["chain_seed"] + 1)
     barrier()
     clocks = clk.stop()
-    loop_ms, prune_ms, launches = ctx.mpcgs_last_timing()
-    t = torch.tensor([loop_ms, prune_ms], dtype=torch.float64, device="cuda")
+    tm = ctx.mpcgs_last_timing_ex()
+    launches = tm["launches"]
+    t = torch.tensor([tm["loop"], tm["prune"], tm["propose"], tm["draw"]], dtype=torch.float64, device="cuda")
     if dist is not None:
         dist.all_reduce(t, op=dist.ReduceOp.MAX)
-    loop_ms, prune_ms = float(t[0]), float(t[1])
+    loop_ms, prune_ms, propose_ms, draw_ms = (float(x) for x in t)
     partials = N * L * (n - 1) * args.steps
     value = partials / (loop_ms / 1e3)
     ms_per_step = loop_ms / args.steps
@@ -361,14 +438,20 @@ def main():
     flops_launch = local_trees * L_scored * (flops_per_site_gm(n) if gm else flops_per_site(n))
     prune_avg_s = (prune_ms / 1e3) / args.steps
     achieved = flops_launch / prune_avg_s / 1e12
-    roof = {"bound": "alu", "achieved": achieved, "peak": pk[args.precision], "unit": "TFLOP/s",
-            "frac": achieved / pk[args.precision],
-            "traffic": traffic_from_profiles(f"{args.workload}_fp{args.precision}" + (f"_{args.model}" if gm else "")),
+    tag = f"{args.workload}_fp{args.precision}" + (f"_{args.model}" if gm else "")
+    roof = {"bound": "alu", "achieved": achieved, "peak": alu[args.precision], "unit": "TFLOP/s",
+            "frac": achieved / alu[args.precision],
+            "peak_source": f"measured: FP{args.precision} FMA microbenchmark on this GPU (mpcgs_probe_peak, "
+                           "csrc/probe.cu), best of 5 before the timed region",
+            "peak_derived": pk[args.precision], "frac_of_derived": achieved / pk[args.precision],
+            "peak_derived_source": f"148 SM x {'64 FP64' if args.precision == 64 else '128 FP32'} FMA lanes x 2 x "
+                                   f"{mhz:.0f} MHz (MEASURED_PEAKS sm_max_mhz)",
+            "lds_peak_measured_gbs": alu["lds_gbs"],
+            "pipe": pipe_from_profiles(tag),
+            "traffic": traffic_from_profiles(tag),
             "kernel": ("k_prune (flat, base-set tips)" if args.ambiguity > 0 else "k_prune_tab")
                       + (" + general model (F84/HKY85)" if gm else ""),
             "prune_share_of_step": prune_ms / loop_ms,
-            "peak_source": f"derived: 148 SM x {'64 FP64' if args.precision == 64 else '128 FP32'} FMA lanes x 2 x "
-                           f"{mhz:.0f} MHz (MEASURED_PEAKS sm_max_mhz)",
             "partials_per_s_prune_only": N * L * (n - 1) / (prune_avg_s * world) if world == 1 else
             local_trees * L * (n - 1) / prune_avg_s}
     if args.compress:
@@ -431,12 +514,24 @@ def main():
         incr = {"proposals_per_s": N * args.steps / (l3 / 1e3), "ms_per_step": l3 / args.steps,
                 "partials_equiv_per_s": partials / (l3 / 1e3), "score_kernel_share": s3 / l3,
                 "speedup_vs_full": loop_ms / l3, "kernel": "k_score_incr"}
+        # k_score_incr reads the generator's stored partials of the three children and of the
+        # ancestors' siblings (36 B per node and site in FP64), mostly from L2: ncu puts it on
+        # the FP64 pipe (latency-bound), not on HBM.  Reported: its HBM fraction from ncu's
+        # DRAM bytes of the same launch over the live launch time, and the ncu pipe numbers.
+        tag3 = f"{args.workload}_fp{args.precision}_incr"
+        tb = traffic_from_profiles(tag3)
+        hbm = float(mp.get("hbm_gbs", 6650.0))
+        if tb:
+            ach = tb / ((s3 / 1e3) / args.steps) / 1e9
+            incr["roofline"] = {"bound": "alu", "hbm_achieved_gbs": ach, "hbm_peak_gbs": hbm, "hbm_frac": ach / hbm,
+                                "traffic": tb, "pipe": pipe_from_profiles(tag3),
+                                "note": "the stored partials are L2-resident between steps; the FP64 pipe "
+                                        "(ncu, 'pipe') is the binding unit, as for full pruning",
+                                "hbm_peak_source": "MEASURED_PEAKS.json hbm_gbs" if "hbm_gbs" in mp else "fallback"}
 
     cpu = None
     if rank == 0 and world == 1 and args.cpu_seconds > 0:
-        v, st, dt = cpu_oracle_sample(wl, args.cpu_seconds, model=args.model, kappa=args.kappa)
-        cpu = {"value": v, "unit": UNIT, "cores": 1, "kind": "oracle",
-               "sample": f"{st} oracle GMH steps with 1 proposal each over all {L} sites ({dt:.1f} s)"}
+        cpu = cpu_baselines(wl, args.cpu_seconds, args.model, args.kappa)
 
     if rank == 0:
         line = {
@@ -445,6 +540,10 @@ def main():
             "vs_baseline": None, "dtype": "f64" if args.precision == 64 else "f32", "data": "synthetic",
             "config": workload_config(args, wl), "proposals_per_s": N * args.steps / (loop_ms / 1e3),
             "roofline": roof, "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": int(launches),
+            "phases_ms_per_step": {"context+propose": propose_ms / args.steps, "prune": prune_ms / args.steps,
+                                   "exchange+draw+commit": draw_ms / args.steps,
+                                   "source": "CUDA events around each phase of every timed step "
+                                             "(mpcgs_last_timing_ex)"},
             "incremental_rescoring": incr,
             "clocks": clocks,
         }

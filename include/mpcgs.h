@@ -263,6 +263,19 @@ mpcgs_status mpcgs_set_timing(mpcgs_ctx* ctx, int32_t on);
 mpcgs_status mpcgs_last_timing(const mpcgs_ctx* ctx, double* loop_ms, double* prune_ms,
                                int64_t* launches);
 
+/* Per-phase device times (ms) of the last device-timed mpcgs_sample loop (timing mode bit 0),
+ * summed over its steps, from the same CUDA events: ms4[0] the loop, [1] context + proposal
+ * resimulation (k_context / k_propose), [2] pruning, [3] record exchange + weights/draws/commit
+ * (k_draw, k_commit_incr).  ms4: host [4]; launches nullable. */
+mpcgs_status mpcgs_last_timing_ex(const mpcgs_ctx* ctx, double* ms4, int64_t* launches);
+
+/* [measurement] Microbenchmarked peak of this GPU for the roofline of the ALU-bound pruning
+ * kernels: kind 0 = FP64 FMA throughput (TFLOP/s, FMA = 2 flops), 1 = FP32 FMA
+ * (TFLOP/s), 2 = shared-memory load bandwidth (GB/s, ld.shared.v4).  Best of 5 launches of
+ * 8 CTAs x 256 threads per SM on the current device, timed with CUDA events (~5 ms each).
+ * No context needed.  MPCGS_E_ARG on a bad kind or NULL value. */
+mpcgs_status mpcgs_probe_peak(int32_t kind, double* value);
+
 const char* mpcgs_last_error(const mpcgs_ctx* ctx);
 void mpcgs_free(mpcgs_ctx* ctx);
 

@@ -9,6 +9,7 @@
 // bracket with device reductions.
 #include <dlfcn.h>
 #include <nccl.h>
+#include <nvtx3/nvToolsExt.h>  // header-only NVTX v3: ranges show in nsys / ncu --nvtx
 
 #include <algorithm>
 #include <chrono>
@@ -82,7 +83,7 @@ struct mpcgs_ctx {
     ncclComm_t comm = nullptr;
     int timing = 0;              // bit 0: events per step / prune launch; bit 1: flush L2 between steps
     void* flush_buf = nullptr;   // 256 MiB scratch written between timed steps (> 126 MB L2)
-    double loop_ms = 0.0, prune_ms = 0.0;
+    double loop_ms = 0.0, prune_ms = 0.0, propose_ms = 0.0, draw_ms = 0.0;
     int graph_steps = 32;
     int64_t launches = 0;
     std::vector<cudaEvent_t> evpool;
@@ -100,6 +101,12 @@ struct mpcgs_ctx {
 };
 
 namespace {
+
+// NVTX range for the duration of an entry point (tracing)
+struct NvtxRange {
+    explicit NvtxRange(const char* name) { nvtxRangePushA(name); }
+    ~NvtxRange() { nvtxRangePop(); }
+};
 
 mpcgs_status fail(mpcgs_ctx* c, mpcgs_status st, const std::string& msg) {
     if (c) {
@@ -1044,6 +1051,7 @@ struct InitTrace {  // MPCGS_TRACE_INIT=1: wall-clock phases of mpcgs_init on st
 };
 
 mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, double theta0, mpcgs_ctx** out) {
+    NvtxRange nvtx_("mpcgs_init");
     InitTrace tr;
     if (!out) return MPCGS_E_ARG;
     *out = nullptr;
@@ -1386,7 +1394,7 @@ mpcgs_status sample_begin(mpcgs_ctx* c, int32_t N, int64_t M, uint64_t seed) {
     if (st) return st;
     CU(cudaMemsetAsync(c->s.counters, 0, 8 * 8, c->work));
     c->launches = 0;
-    c->prune_ms = 0.0;
+    c->prune_ms = c->propose_ms = c->draw_ms = 0.0;
     auto one_step = [&]() -> mpcgs_status {
         mpcgs_status s2 = step_local_launch(c, seed, -1, N, nullptr, nullptr, false);
         if (s2) return s2;
@@ -1427,16 +1435,22 @@ mpcgs_status sample_begin(mpcgs_ctx* c, int32_t N, int64_t M, uint64_t seed) {
             CU(cudaEventRecord(c->evpool[4 * k + 3], c->work));
         }
         CU(cudaEventSynchronize(c->evpool[4 * (steps - 1) + 3]));
-        double tot = 0.0, pr = 0.0;
+        double tot = 0.0, pr = 0.0, pp = 0.0, dr = 0.0;
         for (int64_t k = 0; k < steps; ++k) {
-            float t = 0.f, q = 0.f;
+            float t = 0.f, q = 0.f, p0 = 0.f, d0 = 0.f;
             CU(cudaEventElapsedTime(&t, c->evpool[4 * k + 0], c->evpool[4 * k + 3]));
+            CU(cudaEventElapsedTime(&p0, c->evpool[4 * k + 0], c->evpool[4 * k + 1]));
             CU(cudaEventElapsedTime(&q, c->evpool[4 * k + 1], c->evpool[4 * k + 2]));
+            CU(cudaEventElapsedTime(&d0, c->evpool[4 * k + 2], c->evpool[4 * k + 3]));
             tot += t;
             pr += q;
+            pp += p0;
+            dr += d0;
         }
         c->loop_ms = tot;
         c->prune_ms = pr;
+        c->propose_ms = pp;
+        c->draw_ms = dr;
     } else {
         // CUDA graph of up to graph_steps steps, replayed; the kernels read the step
         // counter from device memory, so one graph serves every step
@@ -1510,6 +1524,7 @@ mpcgs_status sample_end(mpcgs_ctx* c) {
 extern "C" {
 
 mpcgs_status mpcgs_sample(mpcgs_ctx* c, int32_t N, int64_t M, uint64_t seed) {
+    NvtxRange nvtx_("mpcgs_sample");
     mpcgs_status st = sample_begin(c, N, M, seed);
     if (st) return st;
     return sample_end(c);
@@ -1533,6 +1548,16 @@ mpcgs_status mpcgs_sample_loci(mpcgs_ctx* const* ctxs, int32_t n_loci, int32_t N
     return first;
 }
 
+
+mpcgs_status mpcgs_last_timing_ex(const mpcgs_ctx* c, double* ms4, int64_t* launches) {
+    if (!c || !ms4) return MPCGS_E_ARG;
+    ms4[0] = c->loop_ms;
+    ms4[1] = c->propose_ms;
+    ms4[2] = c->prune_ms;
+    ms4[3] = c->draw_ms;
+    if (launches) *launches = c->launches;
+    return MPCGS_OK;
+}
 
 mpcgs_status mpcgs_last_timing(const mpcgs_ctx* c, double* loop_ms, double* prune_ms, int64_t* launches) {
     if (!c) return MPCGS_E_ARG;
@@ -1580,6 +1605,7 @@ mpcgs_status mpcgs_load_samples(mpcgs_ctx* c, int64_t count, const double* S, co
 
 mpcgs_status mpcgs_score_trees(mpcgs_ctx* c, int32_t n_trees, const int32_t* parent, const double* age,
                                double* logL_out) {
+    NvtxRange nvtx_("mpcgs_score_trees");
     CHECK_CTX(c);
     if (n_trees < 0 || (n_trees > 0 && (!parent || !age || !logL_out))) return fail(c, MPCGS_E_ARG, "score_trees args");
     mpcgs_status st = enter(c);
@@ -1663,6 +1689,7 @@ mpcgs_status mpcgs_step_finish(mpcgs_ctx* c, int64_t step, int32_t N, int32_t K,
 
 mpcgs_status mpcgs_step_trace(mpcgs_ctx* c, int64_t step, int32_t N, int32_t K, uint64_t seed, int32_t* target,
                               double* logL, double* S, double* t12, int32_t* pair, int32_t* draws) {
+    NvtxRange nvtx_("mpcgs_step_trace");
     CHECK_CTX(c);
     if (c->world != 1) return fail(c, MPCGS_E_STATE, "step_trace needs world = 1 (use step_local/finish)");
     if (N < 1 || N > c->Nmax || K < 1 || K > N || step < 0) return fail(c, MPCGS_E_ARG, "step_trace args");
@@ -1700,6 +1727,7 @@ mpcgs_status mpcgs_set_theta0(mpcgs_ctx* c, double theta0) {
 
 mpcgs_status mpcgs_em(mpcgs_ctx* c, int32_t n_iter, int32_t N, int64_t M, uint64_t seed, int32_t G,
                       double* theta_trace) {
+    NvtxRange nvtx_("mpcgs_em");
     CHECK_CTX(c);
     if (n_iter < 1 || M < 1) return fail(c, MPCGS_E_ARG, "em: n_iter and n_samples must be positive");
     for (int32_t it = 0; it < n_iter; ++it) {
@@ -1922,6 +1950,7 @@ mpcgs_status estimate_theta_impl(mpcgs_ctx* const* cs, int K, double* theta_hat,
 extern "C" {
 
 mpcgs_status mpcgs_estimate_theta(mpcgs_ctx* c, double* theta_hat, int32_t G, double* grid_theta, double* grid_logL) {
+    NvtxRange nvtx_("mpcgs_estimate_theta");
     CHECK_CTX(c);
     return estimate_theta_impl(&c, 1, theta_hat, G, grid_theta, grid_logL);
 }

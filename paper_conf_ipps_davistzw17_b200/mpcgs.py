@@ -83,6 +83,8 @@ _SIGS = {
     "mpcgs_em_loci": (_i32, [_P, _i32, _i32, _i32, _i64, _P, _i32, _P]),
     "mpcgs_set_timing": (_i32, [_P, _i32]),
     "mpcgs_last_timing": (_i32, [_P, _P, _P, _P]),
+    "mpcgs_last_timing_ex": (_i32, [_P, _P, _P]),
+    "mpcgs_probe_peak": (_i32, [_i32, _P]),
     "mpcgs_last_error": (ctypes.c_char_p, [_P]),
     "mpcgs_free": (None, [_P]),
     "mpcgs_shard_range": (_i32, [_i32, _i32, _i32, _P, _P]),
@@ -263,6 +265,15 @@ def mpcgs_em_loci(contexts, n_iter, n_proposals, n_samples, seeds, n_grid=256):
     _loci_err(lib().mpcgs_em_loci(hs, len(contexts), n_iter, n_proposals, n_samples, _ptr(sd), n_grid,
                                   _ptr(trace)), contexts, "em_loci")
     return trace
+
+
+def mpcgs_probe_peak(kind):
+    """Measured FP64 FMA (0, TFLOP/s), FP32 FMA (1, TFLOP/s) or shared-memory load (2, GB/s) peak."""
+    v = ctypes.c_double()
+    st = lib().mpcgs_probe_peak(int(kind), ctypes.byref(v))
+    if st:
+        raise MpcgsError(st, "probe_peak")
+    return v.value
 
 
 def mpcgs_nccl_unique_id():
@@ -452,6 +463,13 @@ class Context:
     def mpcgs_set_timing(self, mode):
         """mode bit 0: CUDA events per step / kernel; bit 1: 256 MiB L2 flush between steps."""
         self._chk(lib().mpcgs_set_timing(self.h, int(mode) & 3), "set_timing")
+
+    def mpcgs_last_timing_ex(self):
+        """{loop, propose, prune, draw} ms of the last device-timed loop, and its launches."""
+        ms = np.zeros(4)
+        n = ctypes.c_int64()
+        self._chk(lib().mpcgs_last_timing_ex(self.h, _ptr(ms), ctypes.byref(n)), "last_timing_ex")
+        return dict(loop=ms[0], propose=ms[1], prune=ms[2], draw=ms[3], launches=n.value)
 
     def mpcgs_last_timing(self):
         a, b, c = ctypes.c_double(), ctypes.c_double(), ctypes.c_int64()
