@@ -739,14 +739,17 @@ __host__ __device__ size_t tab_smem_bytes(int nops, int need, int trip_cap) {
 #else
 #define MPCGS_TAB_BOUNDS __launch_bounds__(PRUNE_THREADS)
 #endif
+// One CTA scores genealogy `tree` over site tile `tile`; its schedule is gop / ge
+// (global memory written by k_propose); smem_raw = the
+// dynamic shared memory of tab_smem_bytes.
 template <typename T, int DR, int SI, bool PT, int DMX, bool W, bool GM>
-__global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
+__device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int tile, const uint32_t* gop,
+                                               const typename Traits<T>::E4* ge, unsigned char* smem_raw) {
     using E4 = typename Traits<T>::E4;
     using CD = Codes<SI>;
     constexpr uint32_t TABE = PT ? 32u : 16u;  // table entries per tip
     constexpr int BATCH = CD::BATCH;  // sites per batch
     constexpr size_t OPB = GM ? 32 * sizeof(T) : sizeof(E4);  // branch data bytes per op
-    extern __shared__ __align__(16) unsigned char smem_raw[];
     const int nops = a.nops, n = nops + 1;
     const int trip_cap = PT ? a.trip_cap : 0;
     E4* s_e = reinterpret_cast<E4*>(smem_raw);  // F81: {e_a, em_a, e_b, em_b} per op
@@ -766,12 +769,9 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
     __shared__ int s_nc;  // compacted op count
 
     const int tid = threadIdx.x;
-    const int tree = blockIdx.y;
-    const int tile = blockIdx.x;
     int s_begin, s_end;
     tile_range(a, tile, s_begin, s_end);
     const int nb = (s_end - s_begin + BATCH - 1) / BATCH;
-    if (a.tree_need && a.tree_need[tree] > a.need_cap) return;  // deeper tree: scored by the flat pass
 
     auto issue = [&](int b, int buf) {
         const int site0 = s_begin + b * BATCH;
@@ -787,8 +787,6 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
     if (nb > 0) issue(0, 0);
 
     // 1. schedule, branch data and the per-child bounds d (mark_checks, fusion guard)
-    const uint32_t* __restrict__ gop = a.sched_op + (size_t)tree * nops;
-    const E4* __restrict__ ge = reinterpret_cast<const E4*>(a.sched_e) + (size_t)tree * nops;
     const T pi[4] = {(T)a.pi[0], (T)a.pi[1], (T)a.pi[2], (T)a.pi[3]};
     const T pimin = min(min(pi[0], pi[1]), min(pi[2], pi[3]));
     uint32_t* s_code = reinterpret_cast<uint32_t*>(s_tl);  // original codes (s_tl is filled after the scan)
@@ -1124,6 +1122,16 @@ __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
     exact_commit<PRUNE_THREADS>(ex, a.tree_acc + 4 * (size_t)tree, a.tile_cnt + tree, a.tiles,
                                 a.out + (size_t)(a.out_first + tree) * a.out_stride,
                                 reinterpret_cast<unsigned long long*>(s_cod));
+}
+
+template <typename T, int DR, int SI, bool PT, int DMX, bool W, bool GM>
+__global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
+    extern __shared__ __align__(16) unsigned char smem_raw[];
+    const int tree = blockIdx.y;
+    if (a.tree_need && a.tree_need[tree] > a.need_cap) return;  // deeper tree: scored by the flat pass
+    prune_tab_body<T, DR, SI, PT, DMX, W, GM>(
+        a, tree, blockIdx.x, a.sched_op + (size_t)tree * a.nops,
+        reinterpret_cast<const typename Traits<T>::E4*>(a.sched_e) + (size_t)tree * a.nops, smem_raw);
 }
 
 template <typename T, int D, bool W, bool GM, bool AMB>
