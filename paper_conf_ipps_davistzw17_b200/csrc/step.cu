@@ -26,7 +26,7 @@ __global__ void __launch_bounds__(CTX_THREADS) k_context(DevState s, uint64_t se
 
 size_t context_smem_bytes(int n) {
     return sizeof(double) * ((size_t)(n - 1) + n + (n + 1) + (n + 2) + 6 * n + 3 * (n + 1)) +
-           sizeof(int) * (n + 1) + 16;
+           sizeof(int) * ((n + 1) + (2 * (size_t)n - 1) + 2 * (size_t)(n - 1)) + 16;
 }
 
 cudaError_t launch_context(const DevState& s, uint64_t seed, int64_t step, cudaStream_t st) {

@@ -48,6 +48,34 @@ inline __device__ double what(int k, int kk, double len, int l, double theta, bo
     return c3 * c2 * (a - b) / (r2 - r1);
 }
 
+// All six weights of one interval, rows (1,1) (2,2) (2,1) (3,3) (3,2) (3,1), with the
+// expressions of what() (the shared exponentials evaluated once).  One thread computes
+// a whole row: threads of a warp follow one instruction stream (what() per (interval,
+// row) diverged six ways and serialised the transcendentals).
+__device__ __forceinline__ void what_row(double len, int l, double theta, bool inf, double* W) {
+    if (inf) {  // unbounded root interval: only transitions ending at k = 1 (S9)
+        W[0] = 1.0; W[1] = 0.0; W[2] = 1.0; W[3] = 0.0; W[4] = 0.0; W[5] = 1.0;
+        return;
+    }
+    const double r1 = (2.0 * l) / theta;
+    const double r2 = (2.0 + 4.0 * l) / theta;
+    const double r3 = (6.0 + 6.0 * l) / theta;
+    const double c2 = 2.0 / theta, c3 = 6.0 / theta;
+    const double e21 = exp(-(r2 - r1) * len);
+    const double m21 = -expm1(-(r2 - r1) * len);
+    const double e31 = exp(-(r3 - r1) * len);
+    const double m32 = -expm1(-(r3 - r2) * len);
+    const double m31 = -expm1(-(r3 - r1) * len);
+    W[0] = 1.0;
+    W[1] = e21;
+    W[2] = c2 * m21 / (r2 - r1);
+    W[3] = e31;
+    W[4] = c3 * e21 * m32 / (r3 - r2);
+    const double a = m31 / (r3 - r1);
+    const double b = e21 * m32 / (r3 - r2);
+    W[5] = c3 * c2 * (a - b) / (r2 - r1);
+}
+
 // count of x[0..len) <= v (x sorted ascending)
 __device__ __forceinline__ int upper_count(const double* x, int len, double v) {
     int lo = 0, hi = len;
@@ -111,6 +139,9 @@ __device__ void context_body(const DevState& s, uint64_t seed, int64_t step_arg,
     double* sW = sTau + n + 2;        // [n][6] W^ rows: (1,1) (2,2) (2,1) (3,3) (3,2) (3,1)
     double* sBeta = sW + 6 * n;       // [(n+1)][3]
     int* sEntry = reinterpret_cast<int*>(sBeta + 3 * (n + 1));  // [n+1]
+    int* sPar = sEntry + n + 1;       // [nn] parents, staged: tid 0's lookups below hit shared memory
+    int* sLI = sPar + nn;             // [n-1] children of interior nodes (index v - n)
+    int* sRI = sLI + nint;            // [n-1]
     __shared__ int sh[16];
     __shared__ double shd[8];
     __shared__ int s_warp[NT / 32];
@@ -118,8 +149,11 @@ __device__ void context_body(const DevState& s, uint64_t seed, int64_t step_arg,
 
     for (int i = tid; i < nint; i += NT) {
         sAge[i] = s.age[n + i];
+        sLI[i] = s.left[n + i];
+        sRI[i] = s.right[n + i];
         if (s.parent[n + i] < 0) sh[10] = n + i;  // root
     }
+    for (int i = tid; i < nn; i += NT) sPar[i] = s.parent[i];
     __syncthreads();
     if (tid == 0) {
         const int64_t step = step_of(s, step_arg);
@@ -128,11 +162,12 @@ __device__ void context_body(const DevState& s, uint64_t seed, int64_t step_arg,
         U4 w = philox(U4{0u, 0u, (uint32_t)step, TAG_TARGET}, (uint32_t)seed, (uint32_t)(seed >> 32));
         int T = n + (int)__umulhi(w.x, (uint32_t)(n - 2));
         if (T >= root) ++T;
-        const int Par = s.parent[T];
-        const int A = s.parent[Par];
-        const int sib = s.left[Par] == T ? s.right[Par] : s.left[Par];
-        int c[3] = {s.left[T], s.right[T], sib};
-        double a[3] = {s.age[c[0]], s.age[c[1]], s.age[c[2]]};
+        const int Par = sPar[T];
+        const int A = sPar[Par];
+        const int sib = sLI[Par - n] == T ? sRI[Par - n] : sLI[Par - n];
+        int c[3] = {sLI[T - n], sRI[T - n], sib};
+        auto age_of = [&](int v) { return v < n ? 0.0 : sAge[v - n]; };  // tips at age 0 (S22)
+        double a[3] = {age_of(c[0]), age_of(c[1]), age_of(c[2])};
         // sort the three children by (age, id)
         for (int i = 0; i < 3; ++i)
             for (int j = i + 1; j < 3; ++j)
@@ -143,7 +178,7 @@ __device__ void context_body(const DevState& s, uint64_t seed, int64_t step_arg,
         sh[0] = T; sh[1] = Par; sh[2] = A; sh[3] = A < 0; sh[4] = (a[2] == a[1]) ? 3 : 2;
         sh[6] = c[0]; sh[7] = c[1]; sh[8] = c[2];
         shd[0] = a[0]; shd[1] = a[1]; shd[2] = a[2];
-        shd[3] = A < 0 ? CUDART_INF : s.age[A];
+        shd[3] = A < 0 ? CUDART_INF : sAge[A - n];
     }
     __syncthreads();
     MPCGS_TS(6);
@@ -205,24 +240,18 @@ __device__ void context_body(const DevState& s, uint64_t seed, int64_t step_arg,
     MPCGS_TS(8);
     // per-interval bookkeeping and closed-form weights: one thread per (interval,
     // weight), 6 weights per interval (the transcendentals dominate)
-    for (int q = tid; q < 6 * m; q += NT) {
-        const int p = q / 6, w = q - 6 * p;
+    for (int p = tid; p < m; p += NT) {
         const double tp = sTau[p];
         const bool inf = rootcase && p == m - 1;
         const double len = inf ? CUDART_INF : sTau[p + 1] - tp;
         const int fixed_below = upper_count(sF, nfixed, tp);
         const int kids_below = (shd[0] <= tp) + (a1 <= tp) + (a2 <= tp);
         const int l = n - fixed_below - kids_below;
-        if (w == 0) {
-            s.tau[p] = tp;
-            s.len[p] = len;
-            s.lcnt[p] = l;
-            sEntry[p] = (p >= 1 && has3 && tp == a2) ? 1 : 0;
-        }
-        // rows (1,1) (2,2) (2,1) (3,3) (3,2) (3,1)
-        const int k = w == 0 ? 1 : (w < 3 ? 2 : 3);
-        const int kk = w == 0 ? 1 : (w == 1 ? 2 : (w == 2 ? 1 : (w == 3 ? 3 : (w == 4 ? 2 : 1))));
-        sW[p * 6 + w] = what(k, kk, len, l, s.theta0, inf);
+        s.tau[p] = tp;
+        s.len[p] = len;
+        s.lcnt[p] = l;
+        sEntry[p] = (p >= 1 && has3 && tp == a2) ? 1 : 0;
+        what_row(len, l, s.theta0, inf, sW + p * 6);  // rows (1,1) (2,2) (2,1) (3,3) (3,2) (3,1)
     }
     if (tid == 0) sEntry[m] = 0;
     __syncthreads();
@@ -274,9 +303,9 @@ __device__ void context_body(const DevState& s, uint64_t seed, int64_t step_arg,
         s.counters[4] = T;
         if (s.incremental) {  // ancestors of Par and their other children (f2)
             int d = 0, prev = Par;
-            for (int a = sh[2]; a >= 0; a = s.parent[a]) {
+            for (int a = sh[2]; a >= 0; a = sPar[a]) {
                 s.path[d] = a;
-                s.pathsib[d] = s.left[a] == prev ? s.right[a] : s.left[a];
+                s.pathsib[d] = sLI[a - n] == prev ? sRI[a - n] : sLI[a - n];
                 prev = a;
                 ++d;
             }
@@ -526,6 +555,22 @@ __device__ __forceinline__ void propose_warp(const DevState& s, uint64_t seed, i
     const double ax = x == c0 ? ac0 : (x == c1 ? ac1 : ac2);
     const double ay = y == c0 ? ac0 : (y == c1 ? ac1 : ac2);
     const double az = z == c0 ? ac0 : (z == c1 ? ac1 : ac2);
+    // the five changed branches x, y, z, T, Par: lanes 0..4 evaluate their branch factors
+    // in lockstep (one exp + expm1 latency), then lane 0 patches the tree
+    __shared__ double sh_e2[4];
+    {
+        const double lp = rootcase ? 0.0 : tAn - t2;
+        const double bt = lane == 0 ? t1 - ax : (lane == 1 ? t1 - ay : (lane == 2 ? t2 - az : (lane == 3 ? t2 - t1 : lp)));
+        double be, bem;
+        branch_data(s.model, u, bt, be, bem);
+        if (lane < 3) {
+            sh_d[2 + 2 * lane] = be;
+            sh_d[3 + 2 * lane] = bem;
+        } else if (lane < 5) {
+            sh_e2[2 * (lane - 3)] = be;
+            sh_e2[2 * (lane - 3) + 1] = bem;
+        }
+    }
     if (lane == 0) {
         // younger new node keeps the target's id, older keeps the parent's (S15)
         sL[T - n] = min(x, y);
@@ -536,19 +581,6 @@ __device__ __forceinline__ void propose_warp(const DevState& s, uint64_t seed, i
         sNeed[Par] = su_need(sNeed[T], sNeed[z]);
         for (int v = A; v >= 0; v = sPar[v]) sNeed[v] = su_need(sNeed[sL[v - n]], sNeed[sR[v - n]]);
         s.tree_need[local] = sNeed[root];
-    } else if (lane == 1) {
-        branch_data(s.model, u, t1 - ax, sh_d[2], sh_d[3]);
-    } else if (lane == 2) {
-        branch_data(s.model, u, t1 - ay, sh_d[4], sh_d[5]);
-    } else if (lane == 3) {
-        branch_data(s.model, u, t2 - az, sh_d[6], sh_d[7]);
-    }
-    __shared__ double sh_e2[4];
-    if (lane == 4) {
-        branch_data(s.model, u, t2 - t1, sh_e2[0], sh_e2[1]);
-    } else if (lane == 5) {
-        const double lp = rootcase ? 0.0 : tAn - t2;
-        branch_data(s.model, u, lp, sh_e2[2], sh_e2[3]);
     }
     // S_G of the proposal: merge of the sorted fixed ages with {t1, t2} (Eq. 18 via
     MPCGS_TP(4);
@@ -735,6 +767,27 @@ __device__ __forceinline__ void draw_body(const DevState& s, uint64_t seed, int6
     MPCGS_TS(3);
     // commit: the last draw generates the next proposal set (Fig. 12)
     const int I = K > 0 ? s.last_draws[K - 1] : 0;
+    __shared__ double s_be[5], s_bem[5];
+    if (I > 0 && tid < 32) {  // the five new branch factors, one lane each, in lockstep
+        const double* r = s.rec + (size_t)I * REC;
+        const int A = s.ctx_i[2];
+        const int c0 = s.ctx_i[6], c1 = s.ctx_i[7], c2 = s.ctx_i[8];
+        const int pair = (int)rec_ld(r + 4);
+        const double t1 = rec_ld(r + 2), t2 = rec_ld(r + 3);
+        const int x = pair == 2 ? c1 : c0;
+        const int y = pair == 0 ? c1 : c2;
+        const int z = pair == 0 ? c2 : (pair == 1 ? c1 : c0);
+        const double lp = A < 0 ? 0.0 : s.age[A] - t2;
+        const double bt = tid == 0 ? t1 - s.age[x]
+                                   : (tid == 1 ? t1 - s.age[y] : (tid == 2 ? t2 - s.age[z] : (tid == 3 ? t2 - t1 : lp)));
+        double be, bem;
+        branch_data(s.model, s.u, bt, be, bem);
+        if (tid < 5) {
+            s_be[tid] = be;
+            s_bem[tid] = bem;
+        }
+    }
+    __syncthreads();
     if (tid == 0 && I > 0) {
         const double* r = s.rec + (size_t)I * REC;
         const int A = s.ctx_i[2];
@@ -755,12 +808,11 @@ __device__ __forceinline__ void draw_body(const DevState& s, uint64_t seed, int6
         s.parent[T] = Par;
         s.age[T] = t1;
         s.age[Par] = t2;
-        branch_data(s.model, u, t1 - s.age[x], s.e[x], s.em[x]);
-        branch_data(s.model, u, t1 - s.age[y], s.e[y], s.em[y]);
-        branch_data(s.model, u, t2 - s.age[z], s.e[z], s.em[z]);
-        branch_data(s.model, u, t2 - t1, s.e[T], s.em[T]);
-        const double lp = A < 0 ? 0.0 : s.age[A] - t2;
-        branch_data(s.model, u, lp, s.e[Par], s.em[Par]);
+        s.e[x] = s_be[0]; s.em[x] = s_bem[0];
+        s.e[y] = s_be[1]; s.em[y] = s_bem[1];
+        s.e[z] = s_be[2]; s.em[z] = s_bem[2];
+        s.e[T] = s_be[3]; s.em[T] = s_bem[3];
+        s.e[Par] = s_be[4]; s.em[Par] = s_bem[4];
         auto nd = [&](int v) { return v < n ? 0 : s.need[v]; };
         s.need[T] = su_need(nd(x), nd(y));
         s.need[Par] = su_need(nd(T), nd(z));
