@@ -165,7 +165,7 @@ struct DevState {
     double* len;       // [n]
     int32_t* lcnt;     // [n]
     int32_t* entry;    // [n+1]
-    double* omega;     // [n][9]: omega_p(k -> k') at (k-1)*3 + k'-1
+    double* omega;     // [n+1][16]: omega_p(k -> k') at (k-1)*3 + k'-1, then r1 r2 r3, expm1 terms
     double* fixed;     // [n] sorted ages of interior nodes other than T, Par
     // proposals
     double* rec;        // [(Nmax+1)][REC]

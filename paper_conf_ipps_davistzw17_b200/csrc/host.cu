@@ -171,7 +171,7 @@ Layout layout(int n, int L, int Nmax, int64_t Mmax, int precision, int increment
     y.len = take(8 * (size_t)(n + 1));
     y.lcnt = take(4 * (size_t)(n + 1));
     y.entry = take(4 * (size_t)(n + 2));
-    y.omega = take(8 * 9 * (size_t)(n + 1));
+    y.omega = take(8 * 16 * (size_t)(n + 1));  // OM_STRIDE doubles per interval (step_body.cuh)
     y.fixed = take(8 * (size_t)n);
     y.rec = take(8 * REC * (size_t)(Nmax + 1));
     y.tree_need = take(4 * (size_t)Nmax);

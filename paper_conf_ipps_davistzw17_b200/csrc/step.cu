@@ -51,7 +51,7 @@ __global__ void __launch_bounds__(32) k_propose(DevState s, uint64_t seed, int64
 
 size_t propose_smem_bytes(int n) {
     const size_t nn = 2 * (size_t)n - 1;
-    return sizeof(int) * (size_t)propose_int_words(n) + sizeof(double) * ((size_t)(n + 2) + (n + 1) + 9 * (n + 1) + 2 * nn);
+    return sizeof(int) * (size_t)propose_int_words(n) + sizeof(double) * ((size_t)(n + 2) + (n + 1) + OM_STRIDE * (n + 1) + 2 * nn);
 }
 
 cudaError_t launch_propose(const DevState& s, uint64_t seed, int64_t step, int slot_first, int count,
@@ -86,7 +86,7 @@ __global__ void __launch_bounds__(NT) k_draw(DevState s, uint64_t seed, int64_t 
 
 cudaError_t launch_draw(const DevState& s, uint64_t seed, int64_t step, int N, int K, int burnin, int64_t M,
                         int64_t total_steps, cudaStream_t st) {
-    const size_t smem = std::max(sizeof(double) * (size_t)(N + 1), context_smem_bytes(s.n));
+    const size_t smem = std::max(3 * sizeof(double) * (size_t)(N + 1), context_smem_bytes(s.n));
     static size_t attr_bytes = 48 * 1024;
     if (smem > attr_bytes) {
         cudaError_t e = cudaFuncSetAttribute(k_draw<128>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);

@@ -20,6 +20,9 @@ static __device__ long long g_tp[8];
 #endif
 
 constexpr int CTX_THREADS = 256;
+// per-interval record of s.omega: [0..8] omega_p(k -> k') at (k-1)*3 + k'-1, [9..11] r1 r2 r3,
+// [12] expm1(-(r2-r1) len), [13] expm1(-(r3-r2) len) (the walk's event placement)
+constexpr int OM_STRIDE = 16;
 constexpr int DRAW_THREADS = 1024;
 
 // ------------------------------------------------------------------ helpers
@@ -27,39 +30,28 @@ __device__ __forceinline__ int64_t step_of(const DevState& s, int64_t step_arg) 
     return step_arg >= 0 ? step_arg : s.counters[0];
 }
 
-// Scaled weight W^_p(k -> kk) of an interval (length len, l inactive lineages):
-// every weight of the interval carries the common factor e^{r_1 len} (S12).
-inline __device__ double what(int k, int kk, double len, int l, double theta, bool inf) {
-    if (inf) return kk == 1 ? 1.0 : 0.0;  // unbounded root interval, l = 0 (S9)
-    const double r1 = (2.0 * l) / theta;
-    const double r2 = (2.0 + 4.0 * l) / theta;
-    const double r3 = (6.0 + 6.0 * l) / theta;
-    const double c2 = 2.0 / theta, c3 = 6.0 / theta;
-    if (k == 1) return kk == 1 ? 1.0 : 0.0;
-    if (k == 2) {
-        if (kk == 2) return exp(-(r2 - r1) * len);
-        if (kk == 1) return c2 * (-expm1(-(r2 - r1) * len)) / (r2 - r1);
-        return 0.0;
-    }
-    if (kk == 3) return exp(-(r3 - r1) * len);
-    if (kk == 2) return c3 * exp(-(r2 - r1) * len) * (-expm1(-(r3 - r2) * len)) / (r3 - r2);
-    const double a = (-expm1(-(r3 - r1) * len)) / (r3 - r1);
-    const double b = exp(-(r2 - r1) * len) * (-expm1(-(r3 - r2) * len)) / (r3 - r2);
-    return c3 * c2 * (a - b) / (r2 - r1);
-}
-
+// Scaled weights W^_p(k -> kk) of an interval (length len, l inactive lineages;
+// SURVEY App. B closed forms): every weight of the interval carries the common factor
+// e^{r_1 len} (S12).
 // All six weights of one interval, rows (1,1) (2,2) (2,1) (3,3) (3,2) (3,1), with the
 // expressions of what() (the shared exponentials evaluated once).  One thread computes
 // a whole row: threads of a warp follow one instruction stream (what() per (interval,
 // row) diverged six ways and serialised the transcendentals).
-__device__ __forceinline__ void what_row(double len, int l, double theta, bool inf, double* W) {
+// rt (nullable) receives what the forward walk's event placement needs (OM_STRIDE
+// layout): r1, r2, r3 and expm1(-(r2-r1) len), expm1(-(r3-r2) len).
+__device__ __forceinline__ void what_row(double len, int l, double theta, bool inf, double* W, double* rt) {
+    const double r1 = (2.0 * l) / theta;
+    const double r2 = (2.0 + 4.0 * l) / theta;
+    const double r3 = (6.0 + 6.0 * l) / theta;
+    if (rt) {
+        rt[0] = r1; rt[1] = r2; rt[2] = r3;
+        rt[3] = inf ? 0.0 : expm1(-(r2 - r1) * len);
+        rt[4] = inf ? 0.0 : expm1(-(r3 - r2) * len);
+    }
     if (inf) {  // unbounded root interval: only transitions ending at k = 1 (S9)
         W[0] = 1.0; W[1] = 0.0; W[2] = 1.0; W[3] = 0.0; W[4] = 0.0; W[5] = 1.0;
         return;
     }
-    const double r1 = (2.0 * l) / theta;
-    const double r2 = (2.0 + 4.0 * l) / theta;
-    const double r3 = (6.0 + 6.0 * l) / theta;
     const double c2 = 2.0 / theta, c3 = 6.0 / theta;
     const double e21 = exp(-(r2 - r1) * len);
     const double m21 = -expm1(-(r2 - r1) * len);
@@ -251,7 +243,7 @@ __device__ void context_body(const DevState& s, uint64_t seed, int64_t step_arg,
         s.len[p] = len;
         s.lcnt[p] = l;
         sEntry[p] = (p >= 1 && has3 && tp == a2) ? 1 : 0;
-        what_row(len, l, s.theta0, inf, sW + p * 6);  // rows (1,1) (2,2) (2,1) (3,3) (3,2) (3,1)
+        what_row(len, l, s.theta0, inf, sW + p * 6, s.omega + p * OM_STRIDE + 9);  // rows (1,1) (2,2) (2,1) (3,3) (3,2) (3,1)
     }
     if (tid == 0) sEntry[m] = 0;
     __syncthreads();
@@ -285,7 +277,7 @@ __device__ void context_body(const DevState& s, uint64_t seed, int64_t step_arg,
         const double* bn = sBeta + (p + 1) * 3;
         const double be1 = en ? bn[1] : bn[0], be2 = en ? bn[2] : bn[1], be3 = en ? 0.0 : bn[2];
         const double* W = sW + p * 6;
-        double* om = s.omega + p * 9;
+        double* om = s.omega + p * OM_STRIDE;
         om[0] = W[0] * be1; om[1] = 0.0;         om[2] = 0.0;
         om[3] = W[2] * be1; om[4] = W[1] * be2;  om[5] = 0.0;
         om[6] = W[5] * be1; om[7] = W[4] * be2;  om[8] = W[3] * be3;
@@ -316,10 +308,11 @@ __device__ void context_body(const DevState& s, uint64_t seed, int64_t step_arg,
 
 
 // ------------------------------------------------------------------ k_propose
-// One event k -> k-1 in [0, len]: density prop. to e^{-delta s}; inverse CDF.
-inline __device__ double place_one(double len, double delta, double u, bool inf) {
+// One event k -> k-1 in [0, len]: density prop. to e^{-delta s}; inverse CDF with
+// em = expm1(-delta len) precomputed by the context (OM_STRIDE record).
+__device__ __forceinline__ double place_one_em(double len, double delta, double em, double u, bool inf) {
     if (inf) return -log(u) / delta;
-    double sv = -log1p(u * expm1(-delta * len)) / delta;
+    double sv = -log1p(u * em) / delta;
     return fmin(fmax(sv, 0.0), len);
 }
 
@@ -405,13 +398,12 @@ inline __device__ Walk forward_walk(const WalkCtx& s, int m, int k0, bool rootca
     Walk w{0.0, 0.0, 0, 0};
     double tt[2] = {0.0, 0.0};
     int k = k0, events = 0;
-    const double th = s.theta0;
     for (int p = 0; p < m && events < 2; ++p) {
         if (p >= 1) k += s.entry[p];
         const bool inf = rootcase && p == m - 1;
-        const int l = s.lcnt[p];
-        const double r1 = (2.0 * l) / th, r2 = (2.0 + 4.0 * l) / th, r3 = (6.0 + 6.0 * l) / th;
-        const double* om = s.omega + p * 9 + (k - 1) * 3;
+        const double* rr = s.omega + p * OM_STRIDE + 9;  // r1 r2 r3 and the expm1 terms (context)
+        const double r1 = rr[0], r2 = rr[1], r3 = rr[2];
+        const double* om = s.omega + p * OM_STRIDE + (k - 1) * 3;
         const double w0 = om[k - 1];
         const double w1 = k >= 2 ? om[k - 2] : 0.0;
         const double w2 = k >= 3 ? om[k - 3] : 0.0;
@@ -434,7 +426,7 @@ inline __device__ Walk forward_walk(const WalkCtx& s, int m, int k0, bool rootca
         if (choice == 1) {
             const double rk = k == 3 ? r3 : (k == 2 ? r2 : r1);
             const double rk1 = k == 3 ? r2 : r1;
-            tt[events] = t0 + place_one(len, rk - rk1, us.next(), inf);
+            tt[events] = t0 + place_one_em(len, rk - rk1, k == 3 ? rr[4] : rr[3], us.next(), inf);
         } else if (choice == 2) {
             const double u1 = us.next(), u2 = us.next();
             double xo, yo;
@@ -480,8 +472,8 @@ __device__ __forceinline__ void propose_warp(const DevState& s, uint64_t seed, i
     int* sPar = sEn + n + 2;       // [nn] parents
     double* sTau = reinterpret_cast<double*>(psm + propose_int_words(n));  // [n+2]
     double* sLen = sTau + n + 2;   // [n+1]
-    double* sOm = sLen + n + 1;    // [9(n+1)]
-    double* sE = sOm + 9 * (n + 1);  // [nn] branch factor above each node (patched for the proposal)
+    double* sOm = sLen + n + 1;    // [OM_STRIDE (n+1)]
+    double* sE = sOm + OM_STRIDE * (n + 1);  // [nn] branch factor above each node (patched for the proposal)
     double* sEm = sE + nn;           // [nn]
     __shared__ double sh_d[8];  // t1, t2, e/em of changed branches
     __shared__ int sh_i[8];
@@ -506,7 +498,7 @@ __device__ __forceinline__ void propose_warp(const DevState& s, uint64_t seed, i
             sLc[i] = s.lcnt[i];
         }
     }
-    for (int i = lane; i < 9 * m; i += 32) sOm[i] = s.omega[i];
+    for (int i = lane; i < OM_STRIDE * m; i += 32) sOm[i] = s.omega[i];
     for (int i = lane; i < nint; i += 32) {
         sL[i] = s.left[n + i];
         sR[i] = s.right[n + i];
@@ -657,10 +649,13 @@ template <int NT>
 __device__ __forceinline__ void draw_body(const DevState& s, uint64_t seed, int64_t step_arg, int N, int K_arg,
                                           int burnin, int64_t M, int64_t total_steps, double* dsm) {
     MPCGS_TS(0);
-    double* sC = dsm;  // [N+1] cumulative weights
+    double* sC = dsm;               // [N+1] cumulative weights
+    double* sLg = dsm + (N + 1);    // [N+1] logL of every slot, staged once (weights, sample store)
+    double* sSg = sLg + (N + 1);    // [N+1] S_G of every slot (sample store)
     __shared__ double s_red[NT / 32];
     __shared__ double s_max;
     __shared__ int s_K, s_store;
+    __shared__ long long s_stored;
     const int tid = threadIdx.x, lane = tid & 31, wid = tid >> 5;
     const int64_t step = step_of(s, step_arg);
     const int nslots = N + 1;
@@ -676,8 +671,14 @@ __device__ __forceinline__ void draw_body(const DevState& s, uint64_t seed, int6
     }
     const int chunk = (nslots + NT - 1) / NT;
     const int i0 = tid * chunk, i1 = min(nslots, i0 + chunk);
+    const int64_t stored0 = tid == 0 ? s.counters[1] : 0;  // issued early (needed after the barrier)
     double mx = -CUDART_INF;
-    for (int i = i0; i < i1; ++i) mx = fmax(mx, i == 0 ? s.gen[0] : rec_ld(s.rec + (size_t)i * REC));
+    for (int i = i0; i < i1; ++i) {
+        const double li = i == 0 ? s.gen[0] : rec_ld(s.rec + (size_t)i * REC);
+        sLg[i] = li;
+        sSg[i] = i == 0 ? s.gen[1] : rec_ld(s.rec + (size_t)i * REC + 1);
+        mx = fmax(mx, li);
+    }
 #pragma unroll
     for (int o = 16; o > 0; o >>= 1) mx = fmax(mx, __shfl_xor_sync(0xffffffffu, mx, o));
     if (lane == 0) s_red[wid] = mx;
@@ -695,12 +696,13 @@ __device__ __forceinline__ void draw_body(const DevState& s, uint64_t seed, int6
             K = 1;  // burn-in: one draw per set, not stored (Fig. 12)
             store = 0;
         } else {
-            const int64_t rem = M - s.counters[1];
+            const int64_t rem = M - stored0;
             K = (int)(rem < N ? rem : N);  // Alg. 1: N draws per set (S17)
             store = 1;
         }
         s_K = K;
         s_store = store;
+        s_stored = stored0;
     }
     __syncthreads();
     MPCGS_TS(1);
@@ -715,7 +717,7 @@ __device__ __forceinline__ void draw_body(const DevState& s, uint64_t seed, int6
     // w_i = exp(logL_i - max): Eq. 31, proportional to P(D|G_i); inclusive scan in slot order
     double run = 0.0;
     for (int i = i0; i < i1; ++i) {
-        run += exp((i == 0 ? s.gen[0] : rec_ld(s.rec + (size_t)i * REC)) - mx);
+        run += exp(sLg[i] - mx);
         sC[i] = run;
     }
     double x = run;
@@ -743,7 +745,7 @@ __device__ __forceinline__ void draw_body(const DevState& s, uint64_t seed, int6
     MPCGS_TS(2);
     const int K = s_K;
     const double total = sC[N];
-    const int64_t stored = s.counters[1];
+    const int64_t stored = s_stored;
     for (int d = tid; d < K; d += NT) {
         const double u = uniform_at(seed, 0u, (uint32_t)step, TAG_DRAW, (uint32_t)d);
         const double xd = u * total;
@@ -756,9 +758,8 @@ __device__ __forceinline__ void draw_body(const DevState& s, uint64_t seed, int6
         s.last_draws[d] = lo;
         if (s_store) {
             const int64_t j = stored + d;
-            const double* r = s.rec + (size_t)lo * REC;
-            s.sS[j] = rec_ld(r + 1);
-            s.sL[j] = rec_ld(r);
+            s.sS[j] = sSg[lo];
+            s.sL[j] = sLg[lo];
             s.sStep[j] = step;
             s.sSlot[j] = lo;
         }
