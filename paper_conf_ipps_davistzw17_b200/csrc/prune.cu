@@ -58,7 +58,11 @@ static size_t tab_bytes_for(int n) {
                              : tab_smem_bytes<T, PRUNE_DR, PRUNE_SI_LARGE, false, GM>(n - 1, cap, 0);
 }
 
+#ifndef MPCGS_TAB_MIN_N
+#define MPCGS_TAB_MIN_N 8  // below 8 tips the table setup costs more than it saves (c1: 41 -> 37 us per step)
+#endif
 bool prune_uses_tables(int n, int precision, bool general_model) {
+    if (n < MPCGS_TAB_MIN_N) return false;
     size_t bytes;
     if (precision == 32) bytes = general_model ? tab_bytes_for<float, true>(n) : tab_bytes_for<float, false>(n);
     else bytes = general_model ? tab_bytes_for<double, true>(n) : tab_bytes_for<double, false>(n);
