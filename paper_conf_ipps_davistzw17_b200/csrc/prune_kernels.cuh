@@ -15,6 +15,7 @@
 // fixed order by the last CTA of each tree (deterministic, P22).
 #pragma once
 #include <algorithm>
+#include <cstdio>
 #include <type_traits>
 
 #include "arith.cuh"
@@ -739,6 +740,13 @@ __host__ __device__ size_t tab_smem_bytes(int nops, int need, int trip_cap) {
 #else
 #define MPCGS_TAB_BOUNDS __launch_bounds__(PRUNE_THREADS)
 #endif
+#ifdef MPCGS_PRUNE_TS  // diagnosis: setup phase cycles of CTA (0, 0), printed once per launch
+static __device__ long long g_pts[8];
+#define PTS(i) do { if (threadIdx.x == 0 && blockIdx.x == 0 && blockIdx.y == 0) g_pts[i] = clock64(); } while (0)
+#else
+#define PTS(i) do { } while (0)
+#endif
+
 // One CTA scores genealogy `tree` over site tile `tile`; its schedule is gop / ge
 // (global memory written by k_propose); smem_raw = the
 // dynamic shared memory of tab_smem_bytes.
@@ -772,6 +780,7 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
     int s_begin, s_end;
     tile_range(a, tile, s_begin, s_end);
     const int nb = (s_end - s_begin + BATCH - 1) / BATCH;
+    PTS(0);
 
     auto issue = [&](int b, int buf) {
         const int site0 = s_begin + b * BATCH;
@@ -816,6 +825,7 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
         if (tid < 16) s_P[nops * 32 + tid] = (tid % 5 == 0) ? T(1) : T(0);  // identity: the root's up branch
     }
     __syncthreads();
+    PTS(2);
     // 2. warp 0: fuse the first trip_cap (TT, TS) pairs, compact the op list and
     //    lay out the tables (exclusive scans over the original ops)
     if (tid < 32) {
@@ -861,6 +871,7 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
         if (tid == 0) s_nc = (int)c_keep;
     }
     __syncthreads();
+    PTS(3);
     const int nops_c = s_nc;
     // 3. sparse checks (FP64): warp 1 walks the bounds while the others build the tables
     unsigned char* s_chk = reinterpret_cast<unsigned char*>(s_tl);  // s_code is dead after the scan
@@ -872,7 +883,10 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
     //    second entry, side b for the top (SS) or the subtree (TS); none (the
     //    identity) for the root.  Stored in the op record in place of the
     //    children's branch data, which the per-site path no longer needs.
-    for (int i = tid; i < nops_c; i += PRUNE_THREADS) {
+    // (warps other than the bound-walking warp 1 share the ops)
+    constexpr int NSCAN = sparse_checks<T>() ? PRUNE_THREADS - 32 : PRUNE_THREADS;
+    const int tscan = (sparse_checks<T>() && tid >= 64) ? tid - 32 : tid;
+    for (int i = tscan; i < nops_c && !(sparse_checks<T>() && tid >= 32 && tid < 64); i += NSCAN) {
         const uint32_t xi = s_opc[i].h.x;
         const int ty = (int)(xi & 3u), sp = (int)((xi >> 2) & 15u);
         const int lvl = (ty == (int)OP_TS) ? sp - 1 : (ty == (int)OP_SS ? sp - 2 : sp);
@@ -896,126 +910,123 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
         s_opc[i].up[0] = up0;
         s_opc[i].up[1] = up1;
     }
-    //    tables, one 4-vector (row) per work item: tip tables P_{.,x}(t) (Eq. 19-20 at an
-    //    indicator tip), cherry rows tip_a(xa) (.) tip_b(xb), and fused-triplet rows
-    //    tip_c(xc) (.) branch(tip_a(xa) (.) tip_b(xb)) for the four xc -- the TS op
-    //    applied to the cherry's vector, as the per-site path computes it
-    for (int idx = tid; idx < nops_c * 16; idx += PRUNE_THREADS) {
-        const int op = idx >> 4, r = idx & 15;
-        const uint4 ox = s_opc[op].h;
-        const uint32_t ty = ox.x & 3u;
-        T* tab = reinterpret_cast<T*>(reinterpret_cast<char*>(s_tab) + (ox.y & ~TAB_CHECK));
-        T va[4], vb[4];
-        if constexpr (GM) {  // tip vectors are columns of P (row X = parent state)
-            const T* Pa = s_P + ox.z * 32;
-            auto col = [](T (&v)[4], const T* P, int x) {
-#pragma unroll
-                for (int X = 0; X < 4; ++X) v[X] = P[X * 4 + x];
-            };
-            if (ty == OP_TT && PT) {
-                col(va, Pa, r >> 2);
-                col(vb, Pa + 16, r & 3);
-#pragma unroll
-                for (int X = 0; X < 4; ++X) va[X] *= vb[X];
-                st4<T>(tab + r * 4, va);
-            } else if (ty == OP_TT && r < 8) {
-                col(va, Pa + (r < 4 ? 0 : 16), r & 3);
-                st4<T>(tab + r * 4, va);
-            } else if (ty == OP_TS && r < 4) {
-                col(va, Pa, r);
-                st4<T>(tab + r * 4, va);
-            } else if (ty == OP_TTT) {  // op o: P_a, P_b; op o+1: P of tip c, P of the cherry's branch
-                const T* Pc = Pa + 32;
-                col(va, Pa, r >> 2);
-                col(vb, Pa + 16, r & 3);
-#pragma unroll
-                for (int X = 0; X < 4; ++X) va[X] *= vb[X];
-                gm_branch<T>(va, Pc + 16);
-#pragma unroll
-                for (int xc = 0; xc < 4; ++xc) {
-                    col(vb, Pc, xc);
-#pragma unroll
-                    for (int X = 0; X < 4; ++X) vb[X] *= va[X];
-                    st4<T>(tab + (r * 4 + xc) * 4, vb);
-                }
-            }
-        } else {
-            const E4 ed = s_e[ox.z];
-            if (ty == OP_TT && PT) {
-                tipvec<T>(va, r >> 2, (T)ed.x, (T)ed.y, pi);
-                tipvec<T>(vb, r & 3, (T)ed.z, (T)ed.w, pi);
-#pragma unroll
-                for (int X = 0; X < 4; ++X) va[X] *= vb[X];
-                st4<T>(tab + r * 4, va);
-            } else if (ty == OP_TT && r < 8) {  // two tip tables: a at [0, 16), b at [16, 32)
-                if (r < 4) tipvec<T>(va, r, (T)ed.x, (T)ed.y, pi);
-                else tipvec<T>(va, r - 4, (T)ed.z, (T)ed.w, pi);
-                st4<T>(tab + r * 4, va);
-            } else if (ty == OP_TS && r < 4) {
-                tipvec<T>(va, r, (T)ed.x, (T)ed.y, pi);
-                st4<T>(tab + r * 4, va);
-            } else if (ty == OP_TTT) {
-                const E4 e1 = s_e[ox.z + 1];
-                tipvec<T>(va, r >> 2, (T)ed.x, (T)ed.y, pi);
-                tipvec<T>(vb, r & 3, (T)ed.z, (T)ed.w, pi);
-#pragma unroll
-                for (int X = 0; X < 4; ++X) va[X] *= vb[X];
-                branch<T>(va, (T)e1.z, (T)e1.w, pi);
-#pragma unroll
-                for (int xc = 0; xc < 4; ++xc) {
-                    tipvec<T>(vb, xc, (T)e1.x, (T)e1.y, pi);
-#pragma unroll
-                    for (int X = 0; X < 4; ++X) vb[X] *= va[X];
-                    st4<T>(tab + (r * 4 + xc) * 4, vb);
-                }
-            }
-        }
-    }
-    __syncthreads();
-    // the check flags are merged into the op codes after the fold pass (which reads
-    // the codes): by the fusion warp below, or by this loop when there is no fusion
-    if constexpr (sparse_checks<T>() && !(PT && MPCGS_FUSE_SS)) {  // ordered before the op loop by the batch barrier
-        for (int op = tid; op < nops_c; op += PRUNE_THREADS)
-            if (s_chk[op]) s_opc[op].h.x |= OP_CHECK;
-    }
-    // 4. cherry / triplet tables: fold each op's up branch into its table, unless
-    //    an entry is small enough to need a rescale (max < 2^-TS): that table
-    //    stays raw and is checked and transformed per site (TAB_CHECK).  A half
-    //    warp (16 lanes, rows r) covers one op, so the flag is one ballot.
+    __syncthreads();  // every op's up branch is in place
+    PTS(4);
+    //    tables, one row per work item: tip tables P_{.,x}(t) (Eq. 19-20 at an indicator
+    //    tip), cherry rows tip_a(xa) (.) tip_b(xb), and fused-triplet rows tip_c(xc) (.)
+    //    branch(tip_a(xa) (.) tip_b(xb)) for the four xc -- the TS op applied to the
+    //    cherry's vector, as the per-site path computes it.
+    // 4. cherry / triplet tables are stored with their op's up branch folded in, unless
+    //    an entry is small enough to need a rescale (max < 2^-TS): that table stays raw
+    //    and is checked and transformed per site (TAB_CHECK).  A half warp (16 lanes,
+    //    rows r) covers one op, so the flag is one ballot; each entry is stored once.
     const int nrow = ((nops_c * 16 + 31) / 32) * 32;
-    for (int idx = tid; idx < nrow && PT; idx += PRUNE_THREADS) {
+    for (int idx = tid; idx < nrow; idx += PRUNE_THREADS) {
         const int op = idx >> 4, r = idx & 15;
-        bool tabop = false, small = false;
-        T* tab = nullptr;
+        bool tabop = false, small = false;  // tabop: a cherry / triplet table to fold (PT)
         int ne = 1;
+        T* tab = nullptr;
+        T v[4][4];
         if (op < nops_c) {
             const uint4 ox = s_opc[op].h;
             const uint32_t ty = ox.x & 3u;
-            tabop = ty == OP_TT || ty == OP_TTT;
-            ne = ty == OP_TTT ? 4 : 1;
-            tab = reinterpret_cast<T*>(reinterpret_cast<char*>(s_tab) + (ox.y & ~TAB_CHECK)) + r * ne * 4;
-            for (int e = 0; e < ne && tabop; ++e) {
-                T v[4];
-                ld4<T>(v, tab + 4 * e);
-                small |= small4(v);
+            tab = reinterpret_cast<T*>(reinterpret_cast<char*>(s_tab) + (ox.y & ~TAB_CHECK));
+            T va[4], vb[4];
+            if constexpr (GM) {  // tip vectors are columns of P (row X = parent state)
+                const T* Pa = s_P + ox.z * 32;
+                auto col = [](T (&w)[4], const T* P, int x) {
+#pragma unroll
+                    for (int X = 0; X < 4; ++X) w[X] = P[X * 4 + x];
+                };
+                if (ty == OP_TT && PT) {
+                    col(va, Pa, r >> 2);
+                    col(vb, Pa + 16, r & 3);
+#pragma unroll
+                    for (int X = 0; X < 4; ++X) v[0][X] = va[X] * vb[X];
+                    tabop = true;
+                } else if (ty == OP_TT && r < 8) {
+                    col(va, Pa + (r < 4 ? 0 : 16), r & 3);
+                    st4<T>(tab + r * 4, va);
+                } else if (ty == OP_TS && r < 4) {
+                    col(va, Pa, r);
+                    st4<T>(tab + r * 4, va);
+                } else if (ty == OP_TTT) {  // op o: P_a, P_b; op o+1: P of tip c, P of the cherry's branch
+                    const T* Pc = Pa + 32;
+                    col(va, Pa, r >> 2);
+                    col(vb, Pa + 16, r & 3);
+#pragma unroll
+                    for (int X = 0; X < 4; ++X) va[X] *= vb[X];
+                    gm_branch<T>(va, Pc + 16);
+#pragma unroll
+                    for (int xc = 0; xc < 4; ++xc) {
+                        col(vb, Pc, xc);
+#pragma unroll
+                        for (int X = 0; X < 4; ++X) v[xc][X] = vb[X] * va[X];
+                    }
+                    tabop = true;
+                    ne = 4;
+                }
+            } else {
+                const E4 ed = s_e[ox.z];
+                if (ty == OP_TT && PT) {
+                    tipvec<T>(va, r >> 2, (T)ed.x, (T)ed.y, pi);
+                    tipvec<T>(vb, r & 3, (T)ed.z, (T)ed.w, pi);
+#pragma unroll
+                    for (int X = 0; X < 4; ++X) v[0][X] = va[X] * vb[X];
+                    tabop = true;
+                } else if (ty == OP_TT && r < 8) {  // two tip tables: a at [0, 16), b at [16, 32)
+                    if (r < 4) tipvec<T>(va, r, (T)ed.x, (T)ed.y, pi);
+                    else tipvec<T>(va, r - 4, (T)ed.z, (T)ed.w, pi);
+                    st4<T>(tab + r * 4, va);
+                } else if (ty == OP_TS && r < 4) {
+                    tipvec<T>(va, r, (T)ed.x, (T)ed.y, pi);
+                    st4<T>(tab + r * 4, va);
+                } else if (ty == OP_TTT) {
+                    const E4 e1 = s_e[ox.z + 1];
+                    tipvec<T>(va, r >> 2, (T)ed.x, (T)ed.y, pi);
+                    tipvec<T>(vb, r & 3, (T)ed.z, (T)ed.w, pi);
+#pragma unroll
+                    for (int X = 0; X < 4; ++X) va[X] *= vb[X];
+                    branch<T>(va, (T)e1.z, (T)e1.w, pi);
+#pragma unroll
+                    for (int xc = 0; xc < 4; ++xc) {
+                        tipvec<T>(vb, xc, (T)e1.x, (T)e1.y, pi);
+#pragma unroll
+                        for (int X = 0; X < 4; ++X) v[xc][X] = vb[X] * va[X];
+                    }
+                    tabop = true;
+                    ne = 4;
+                }
             }
+#pragma unroll
+            for (int e = 0; e < 4; ++e)
+                if (tabop && e < ne) small |= small4(v[e]);
         }
         const unsigned m = __ballot_sync(0xffffffffu, small);
         const bool raw = ((m >> (tid & 16)) & 0xffffu) != 0u;
         if (tabop) {
+            T* row = tab + r * ne * 4;
             if (raw) {
                 if (r == 0) s_opc[op].h.y |= TAB_CHECK;
             } else {
                 const UpBr<T, GM> ub(s_opc[op].up, s_P);
-                for (int e = 0; e < ne; ++e) {
-                    T v[4];
-                    ld4<T>(v, tab + 4 * e);
-                    ub.apply(v, pi);
-                    st4<T>(tab + 4 * e, v);
-                }
+#pragma unroll
+                for (int e = 0; e < 4; ++e)
+                    if (e < ne) ub.apply(v[e], pi);
             }
+#pragma unroll
+            for (int e = 0; e < 4; ++e)
+                if (e < ne) st4<T>(row + 4 * e, v[e]);
         }
     }
+    // the check flags are merged into the op codes after this pass (which reads the
+    // codes): by the fusion warp below, or by this loop when there is no fusion
+    if constexpr (sparse_checks<T>() && !(PT && MPCGS_FUSE_SS)) {  // ordered before the op loop by the batch barrier
+        __syncthreads();
+        for (int op = tid; op < nops_c; op += PRUNE_THREADS)
+            if (s_chk[op]) s_opc[op].h.x |= OP_CHECK;
+    }
+    PTS(5);
     // 5. fuse each folded cherry / triplet op with an SS that immediately merges its
     //    result: one TS-type op at the table op's depth (top (.) table entry) with the
     //    SS's check flag and up branch -- one dispatch, push and pop fewer per pair.
@@ -1059,6 +1070,7 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
         }
         __syncthreads();
         nops_run = s_nc;
+    PTS(6);
     }
 
     SiteAcc<W> acc;
@@ -1119,9 +1131,16 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
         acc.reset();
     }
     // the code staging buffers are free now (the last batch ended with a barrier)
+    PTS(7);
     exact_commit<PRUNE_THREADS>(ex, a.tree_acc + 4 * (size_t)tree, a.tile_cnt + tree, a.tiles,
                                 a.out + (size_t)(a.out_first + tree) * a.out_stride,
                                 reinterpret_cast<unsigned long long*>(s_cod));
+#ifdef MPCGS_PRUNE_TS
+    if (threadIdx.x == 0 && blockIdx.x == 0 && blockIdx.y == 0 && (clock64() & 7) == 0)
+        printf("prune setup: load %lld compact %lld tables %lld fold %lld fuse %lld | batches %lld (nb %d, ops %d)\n",
+               g_pts[2] - g_pts[0], g_pts[3] - g_pts[2], g_pts[4] - g_pts[3], g_pts[5] - g_pts[4], g_pts[6] - g_pts[5],
+               g_pts[7] - g_pts[6], nb, nops_run);
+#endif
 }
 
 template <typename T, int DR, int SI, bool PT, int DMX, bool W, bool GM>

@@ -794,7 +794,7 @@ __device__ __forceinline__ void draw_body(const DevState& s, uint64_t seed, int6
         const int A = s.ctx_i[2];
         const int c0 = s.ctx_i[6], c1 = s.ctx_i[7], c2 = s.ctx_i[8];
         const int pair = (int)rec_ld(r + 4);
-        const double t1 = rec_ld(r + 2), t2 = rec_ld(r + 3), u = s.u;
+        const double t1 = rec_ld(r + 2), t2 = rec_ld(r + 3);
         const int x = pair == 2 ? c1 : c0;
         const int y = pair == 0 ? c1 : c2;
         const int z = pair == 0 ? c2 : (pair == 1 ? c1 : c0);
