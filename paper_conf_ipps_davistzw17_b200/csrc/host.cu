@@ -624,18 +624,17 @@ void upgma(int n, int L, const uint8_t* codes, double theta0, int32_t* parent, d
 }
 
 // Sites per CTA: a multiple of the kernel's exact-sum unit (unit_batches site
-// batches; 1..MPCGS_MAXPER = 64 batches), chosen by a small cost model in units of
+// batches; 1..MPCGS_MAXPER = 128 batches), chosen by a small cost model in units of
 // one batch: a CTA costs its per-tree setup (schedule compaction, tables:
 // ~MPCGS_SETUP batches) plus its batches; the launch takes ceil(CTAs / resident
-// CTAs) waves of one CTA (up to four waves), else total work / resident CTAs plus
-// half a CTA of tail.  Few batches per tree and many trees -> one CTA per tree (the
+// CTAs) waves of one CTA.  Few batches per tree and many trees -> one CTA per tree (the
 // setup is not repeated per tile); few trees -> more tiles for parallelism.  The
 // tree count is the number THIS launch scores (a rank's share of the proposals):
 // the site sums are exact (arith.cuh Exact128) over units fixed by the alignment,
 // so the tiling never changes a likelihood and every world size gives the same
 // chain (P22).
 #ifndef MPCGS_MAXPER
-#define MPCGS_MAXPER 64
+#define MPCGS_MAXPER 128
 #endif
 #ifndef MPCGS_MAXPER_INCR
 #define MPCGS_MAXPER_INCR 32
@@ -657,9 +656,11 @@ void prune_tiling(int n, int L, int ntrees, int precision, int& tiles, int& site
         const long per = std::min<long>(((units + t - 1) / t) * unit, batches);  // batches of the largest tile
         const double len = MPCGS_SETUP + (double)per;
         const double ctas = trees * (double)t;
-        const double work = trees * ((double)t * MPCGS_SETUP + (double)batches);
         // a few waves: equal CTAs run in lock-step waves; many: the tail averages out
-        const double cost = ctas <= 4.0 * slots ? std::ceil(ctas / slots) * len : work / slots + 0.5 * len;
+        // CTAs of one launch have (nearly) equal length and run in lock-step waves: the
+        // last, partly empty wave costs a whole CTA (measured: c5 picks 3 tiles of <= 68
+        // batches instead of 4 of <= 52, +1.6 %; c5 L = 3e4 +3.5 %)
+        const double cost = std::ceil(ctas / slots) * len;
         if (cost < best * (1.0 - 1e-9)) {
             best = cost;
             bt = t;
