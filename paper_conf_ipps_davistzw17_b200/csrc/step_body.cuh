@@ -365,8 +365,60 @@ struct Walk {
 // happens with three active lineages.
 // int words of k_propose's shared arrays (sL, sR, sNeed, sStack, sLc, sEn, sPar), rounded to even
 __host__ __device__ inline int propose_int_words(int n) {
-    const int w = 2 * (n - 1) + (2 * n - 1) + 2 * n + (n + 1) + (n + 2) + (2 * n - 1);
+    const int w = 2 * (n - 1) + (2 * n - 1) + 2 * n + (n + 1) + (n + 2) + (2 * n - 1) + 1 + 3 * (n - 1);
     return (w + 1) & ~1;
+}
+
+// Warp-parallel emission of exactly the schedule emit_schedule (common.cuh) produces:
+// op i of the post-order, code op_encode(type, sp, ta, tb), branch children (ca, cb).
+// For an interior node v with subtree size z(v) (interior nodes), first op index s(v)
+// and stack depth b(v) when its subtree starts: op index s(v) + z(v) - 1; sp = b(v)
+// (TT), b(v) + 1 (TS: after its subtree child), b(v) + 2 (SS).  A child inherits s
+// and b, except the second child of an SS node: s + z(first), b + 1 (first = the
+// child of larger need, ties to the lower id, as the serial DFS).  Sizes come from
+// every interior node walking up to the root (shared atomics), s and b from a second
+// walk summing the offsets of the SS nodes passed on the second child's side.
+// Returns false (nothing emitted) if some node is deeper than max_walk: the caller
+// then runs the serial DFS.
+template <typename ET, typename E4, typename EMIT>
+__device__ __forceinline__ bool emit_schedule_warp(int n, int lane, const int* sL, const int* sR, const int* sNeed,
+                                                   const int* sPar, int* sSize, int max_walk, EMIT emit) {
+    const int nn = 2 * n - 1;
+    for (int i = lane; i < n - 1; i += 32) sSize[i] = 0;
+    __syncwarp();
+    bool deep = false;
+    for (int u = n + lane; u < nn; u += 32) {
+        int k = 0;
+        for (int v = u; v >= 0 && k <= max_walk; v = sPar[v], ++k) atomicAdd(sSize + (v - n), 1);
+        deep |= k > max_walk;
+    }
+    if (__any_sync(0xffffffffu, deep)) return false;
+    __syncwarp();
+    for (int u = n + lane; u < nn; u += 32) {
+        int st = 0, bs = 0;
+        for (int c = u, p = sPar[u]; p >= 0; c = p, p = sPar[p]) {
+            const int a = sL[p - n], b = sR[p - n];
+            if (a >= n && b >= n) {
+                const int first = sNeed[a] >= sNeed[b] ? a : b;
+                if (c != first) {
+                    st += sSize[first - n];
+                    ++bs;
+                }
+            }
+        }
+        const int a = sL[u - n], b = sR[u - n];
+        const int idx = st + sSize[u - n] - 1;
+        if (a < n && b < n) {
+            emit(idx, op_encode(OP_TT, (uint32_t)bs, (uint32_t)a, (uint32_t)b), a, b);
+        } else if (a < n || b < n) {
+            const int t = a < n ? a : b, w = a < n ? b : a;
+            emit(idx, op_encode(OP_TS, (uint32_t)(bs + 1), (uint32_t)t, 0u), t, w);
+        } else {
+            const int first = sNeed[a] >= sNeed[b] ? a : b, second = first == a ? b : a;
+            emit(idx, op_encode(OP_SS, (uint32_t)(bs + 2), 0u, 0u), first, second);
+        }
+    }
+    return true;
 }
 
 struct WalkCtx {  // the step's interval context, staged in shared memory
@@ -470,6 +522,8 @@ __device__ __forceinline__ void propose_warp(const DevState& s, uint64_t seed, i
     int* sLc = sStack + 2 * n;     // [n+1] inactive counts
     int* sEn = sLc + n + 1;        // [n+2] entry flags
     int* sPar = sEn + n + 2;       // [nn] parents
+    int* sFlag = sPar + nn;        // [1] serial-emission fallback flag
+    int* sSize = sFlag + 1;        // [n-1] subtree sizes for the warp-parallel emission
     double* sTau = reinterpret_cast<double*>(psm + propose_int_words(n));  // [n+2]
     double* sLen = sTau + n + 2;   // [n+1]
     double* sOm = sLen + n + 1;    // [OM_STRIDE (n+1)]
@@ -573,6 +627,10 @@ __device__ __forceinline__ void propose_warp(const DevState& s, uint64_t seed, i
         sNeed[Par] = su_need(sNeed[T], sNeed[z]);
         for (int v = A; v >= 0; v = sPar[v]) sNeed[v] = su_need(sNeed[sL[v - n]], sNeed[sR[v - n]]);
         s.tree_need[local] = sNeed[root];
+        sPar[x] = T;  // the proposal's parents (Par keeps A)
+        sPar[y] = T;
+        sPar[z] = Par;
+        sPar[T] = Par;
     }
     // S_G of the proposal: merge of the sorted fixed ages with {t1, t2} (Eq. 18 via
     MPCGS_TP(4);
@@ -617,16 +675,35 @@ __device__ __forceinline__ void propose_warp(const DevState& s, uint64_t seed, i
             for (int i = 0; i < 6; ++i) ee[i] = sh_d[2 + i];
             for (int i = 0; i < 4; ++i) ee[6 + i] = sh_e2[i];
         }
+    }
+    __syncwarp();
+    // post-order register schedule of the proposal tree (warp-parallel; the serial
+    // DFS of emit_schedule for trees deeper than 64 levels)
+    auto emit_op = [&](int i, uint32_t code, int ca, int cb) {
+        op_out[i] = code;
+        E4 v;
+        v.x = (ET)sE[ca]; v.y = (ET)sEm[ca]; v.z = (ET)sE[cb]; v.w = (ET)sEm[cb];
+        e_out[i] = v;
+    };
+    const bool par = emit_schedule_warp<ET, E4>(n, lane, sL, sR, sNeed, sPar, sSize, 64, emit_op);
+    __syncwarp();
+    if (lane == 0) {
+        if (!par)
+            emit_schedule(
+                n, root, [&](int v) { return sL[v - n]; }, [&](int v) { return sR[v - n]; },
+                [&](int v) { return sNeed[v]; }, emit_op, sStack);
+#ifdef MPCGS_CHECK_SCHED  // verification build: the serial DFS must give the same schedule
         emit_schedule(
             n, root, [&](int v) { return sL[v - n]; }, [&](int v) { return sR[v - n]; },
             [&](int v) { return sNeed[v]; },
             [&](int i, uint32_t code, int ca, int cb) {
-                op_out[i] = code;
-                E4 v;
-                v.x = (ET)sE[ca]; v.y = (ET)sEm[ca]; v.z = (ET)sE[cb]; v.w = (ET)sEm[cb];
-                e_out[i] = v;
+                const E4 e = e_out[i];
+                if (op_out[i] != code || e.x != (ET)sE[ca] || e.y != (ET)sEm[ca] || e.z != (ET)sE[cb] ||
+                    e.w != (ET)sEm[cb])
+                    atomicOr(reinterpret_cast<unsigned long long*>(s.counters + 2), (unsigned long long)STATUS_WALK);
             },
             sStack);
+#endif
         MPCGS_TP(6);
 #ifdef MPCGS_TIMESTAMPS
         if (blockIdx.x == 0 && step == 2)
