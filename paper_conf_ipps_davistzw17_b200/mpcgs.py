@@ -285,6 +285,33 @@ def mpcgs_nccl_unique_id():
 
 
 # ------------------------------------------------------------------ context API
+def _config(precision=64, burnin_steps=0, max_proposals=1024, max_samples=1 << 20, base_freq=None, mu=0.0,
+            incremental=False, compress_patterns=False, model="F81", kappa=0.0, ambiguity=False):
+    cfg = mpcgs_config()
+    lib().mpcgs_config_default(ctypes.byref(cfg))
+    if base_freq is not None:
+        for i in range(4):
+            cfg.base_freq[i] = float(base_freq[i])
+    cfg.mu = float(mu)
+    cfg.precision = int(precision)
+    cfg.burnin_steps = int(burnin_steps)
+    cfg.max_proposals = int(max_proposals)
+    cfg.max_samples = int(max_samples)
+    cfg.incremental = int(bool(incremental))
+    cfg.compress_patterns = int(bool(compress_patterns))
+    cfg.model = MODELS[model] if isinstance(model, str) else int(model)
+    cfg.kappa = float(kappa)
+    cfg.ambiguity = int(bool(ambiguity))
+    return cfg
+
+
+def mpcgs_workspace_bytes_cfg(n_seq, n_sites, **options):
+    """Device bytes a context of these capacities / options needs (Context keyword names):
+    a caller-owned workspace of this size can be passed as Context(..., workspace=(ptr, bytes))."""
+    cfg = _config(**options)
+    return int(lib().mpcgs_workspace_bytes_cfg(int(n_seq), int(n_sites), ctypes.byref(cfg)))
+
+
 class Context:
     """Owns an mpcgs_ctx*.  Methods map 1:1 to the C entry points."""
 
@@ -293,21 +320,8 @@ class Context:
                  nccl_id=None, stream=None, workspace=None, phylip=None, incremental=False,
                  compress_patterns=False, model="F81", kappa=0.0, ambiguity=False, init_newick=None):
         L = lib()
-        cfg = mpcgs_config()
-        L.mpcgs_config_default(ctypes.byref(cfg))
-        if base_freq is not None:
-            for i in range(4):
-                cfg.base_freq[i] = float(base_freq[i])
-        cfg.mu = float(mu)
-        cfg.precision = int(precision)
-        cfg.burnin_steps = int(burnin_steps)
-        cfg.max_proposals = int(max_proposals)
-        cfg.max_samples = int(max_samples)
-        cfg.incremental = int(bool(incremental))
-        cfg.compress_patterns = int(bool(compress_patterns))
-        cfg.model = MODELS[model] if isinstance(model, str) else int(model)
-        cfg.kappa = float(kappa)
-        cfg.ambiguity = int(bool(ambiguity))
+        cfg = _config(precision, burnin_steps, max_proposals, max_samples, base_freq, mu, incremental,
+                      compress_patterns, model, kappa, ambiguity)
         self._keep = []
         if init_newick is not None:
             nw = init_newick.encode() if isinstance(init_newick, str) else bytes(init_newick)
