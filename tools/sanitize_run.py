@@ -11,7 +11,7 @@ import paper_conf_ipps_davistzw17_b200 as P  # noqa: E402
 
 for prec in (64, 32):
     for inc in (False, True):
-        for name, over in (("c1", {}), ("c4", {"n": 128, "L": 300, "N": 16})):
+        for name, over in (("c1", {}), ("c3", {"L": 600, "N": 32}), ("c4", {"n": 128, "L": 300, "N": 16})):
             wl = synth.workload(name, **over)
             rows = synth.to_strings(wl["codes"])
             N = wl["N"]
@@ -24,4 +24,18 @@ for prec in (64, 32):
             c.mpcgs_score_trees(np.stack([p, wl["true_parent"]]), np.stack([a, wl["true_age"]]))
             c.free()
             print(name, prec, inc, "theta-hat", th)
+# compressed patterns, virtual ranks (records through the host), loaded samples (a7)
+wl = synth.workload("c2", L=700)
+rows = synth.to_strings(wl["codes"])
+c = P.Context(rows, wl["theta0"], compress_patterns=True, max_proposals=64, max_samples=256)
+c.mpcgs_sample(64, 256, 5)
+r = [P.Context(rows, wl["theta0"], max_proposals=64, max_samples=4, rank=k, world=2) for k in range(2)]
+for k, ck in enumerate(r):
+    ck.mpcgs_step_local(0, 64, 9)
+full = np.concatenate([ck.mpcgs_get_records(*P.mpcgs_shard_range(64, k, 2)) for k, ck in enumerate(r)])
+for ck in r:
+    ck.mpcgs_put_records(1, full)
+    ck.mpcgs_step_finish(0, 64, 64, 9)
+c.mpcgs_load_samples(np.array([1.0, 100.0, 3.0]), 2.15)
+print("bimodal theta-hat", c.mpcgs_estimate_theta(64))
 print("sanitize run done")
