@@ -50,10 +50,11 @@ def flops_per_site(n: int) -> int:
 
 
 def flops_per_site_gm(n: int) -> int:
-    """Same under a general reversible model (F84 / HKY85): a tip
-    child is a column of P (0 flops), an internal child a 4x4 matrix-vector product
-    (16 mul + 12 add), node product 4."""
-    return 28 * (n - 2) + 4 * (n - 1)
+    """Same under F84 / HKY85 with the structured closed form of P(t)
+    (DESIGN.md): a tip child is a column of P (0 flops), an internal child
+    (P v)_i = a T + b_g G_g + c_g v_i -- G_R, G_Y 6, T 1, a T 1, two b_g G_g + a T 4,
+    four c_g v_i + x_g 8 = 20 flops; node product 4."""
+    return 20 * (n - 2) + 4 * (n - 1)
 
 
 def peaks():
@@ -361,8 +362,6 @@ def main():
         over["N"] = args.N
     wl = synth.workload(args.workload, theta_true=args.theta_true, **over)
     if args.ambiguity > 0:  # IUPAC ambiguity codes + gaps (reading S24)
-        import numpy as np
-
         wl["codes"] = synth.ambiguate(wl["codes"], args.ambiguity, np.random.default_rng(wl["chain_seed"] + 7),
                                       gap_frac=args.ambiguity / 2)
     if args.impl == "reference":

@@ -200,7 +200,7 @@ Layout layout(int n, int L, int Nmax, int64_t Mmax, int precision, int increment
     y.iee = take(80 * (size_t)Nmax);
     y.cinfo = take(32);
     y.gen_order = take(4 * (size_t)n);
-    y.gm = take(model ? 8 * 36 : 0);
+    y.gm = take(model ? 8 * 48 : 0);
     y.sched_P = take(model ? 16 * tsz * 2 * (size_t)Nmax * nops : 0);
     y.total = o;
     return y;
@@ -232,6 +232,27 @@ void rate_matrix(int model, double kappa, const double pi[4], double Q[16]) {
     }
     const double scale = flux > 0.0 ? 1.0 / flux : 1.0;
     for (int k = 0; k < 16; ++k) Q[k] *= scale;
+}
+
+// Structured constants of F84 / HKY85 (gm[36..40], read by the table kernel): with
+// the rate matrix normalised by s (rate_matrix), P(t) v has the closed form
+//   (P(t) v)_i = (1 - e^{-s t}) T + (e^{-s t} - e^{-s A_g t}) G_g / Pi_g + e^{-s A_g t} v_i,
+// T = pi . v, G_g = sum_{j in g} pi_j v_j, g = the purine / pyrimidine group of i:
+// Q = s [J + kappa K - (1 + kappa) I] for F84 (J = 1 pi^T, K_ij = [same group] pi_j / Pi_g,
+// commuting projections with JK = KJ = J) gives A_R = A_Y = 1 + kappa; HKY85 gives
+// A_g = 1 + Pi_g (kappa - 1) (Hasegawa, Kishino & Yano 1985).  {s, A_R, A_Y, Pi_R, Pi_Y}.
+void model_consts(int model, double kappa, const double pi[4], double out[5]) {
+    double Q[16];
+    rate_matrix(model, kappa, pi, Q);
+    // rate_matrix scales the unnormalised rates by s: recover s from one off-diagonal entry
+    // (q_01 = s pi_1, a transversion in both models)
+    const double s = Q[0 * 4 + 1] / pi[1];
+    const double PiR = pi[0] + pi[2], PiY = pi[1] + pi[3];
+    out[0] = s;
+    out[1] = model == MPCGS_MODEL_F84 ? 1.0 + kappa : 1.0 + PiR * (kappa - 1.0);
+    out[2] = model == MPCGS_MODEL_F84 ? 1.0 + kappa : 1.0 + PiY * (kappa - 1.0);
+    out[3] = PiR;
+    out[4] = PiY;
 }
 
 // Eigen-system of a reversible Q: S = D^1/2 Q D^-1/2 (D = diag pi) is symmetric;
@@ -1130,7 +1151,7 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
     // substitution model: F81 unless F84 / HKY85 is asked for
     c->model = cfg->model;
     c->kappa = cfg->kappa;
-    double gm[36] = {0};
+    double gm[48] = {0};  // eigen-system [0, 36) (flat kernel, k_pmat) + structured constants [36, 41)
     if (c->model != MPCGS_MODEL_F81) {
         const char* why = nullptr;
         if (c->model != MPCGS_MODEL_F84 && c->model != MPCGS_MODEL_HKY85) why = "unknown substitution model";
@@ -1145,6 +1166,7 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
         double Q[16];
         rate_matrix(c->model, c->kappa, pi, Q);
         eigen_system(Q, pi, gm);
+        model_consts(c->model, c->kappa, pi, gm + 36);
         u = 1.0;  // rates normalised to one substitution per unit time (S3); mu is not used
     }
     // G0

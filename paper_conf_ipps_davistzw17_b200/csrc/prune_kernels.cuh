@@ -114,6 +114,56 @@ __device__ __forceinline__ void gm_branch(T (&R)[4], const T* __restrict__ P) {
     for (int i = 0; i < 4; ++i) R[i] = o[i];
 }
 
+// ---- structured F84 / HKY85 branches (table kernel; host.cu model_consts): a branch
+// of length t is the record C = {a, b_R, b_Y, c_R, c_Y} with
+//   (P(t) v)_i = a T + b_g G_g + c_g v_i,   T = pi . v,  G_g = sum_{j in g} pi_j v_j,
+// a = 1 - e^{-s t}, b_g = (e^{-s t} - e^{-s A_g t}) / Pi_g, c_g = e^{-s A_g t}; purines A, G
+// (0, 2), pyrimidines C, T (1, 3).  12 FP instructions per branch instead of the 16 of a
+// 4x4 matrix-vector product, and 5 values per branch instead of 16.
+constexpr int GMC = 8;  // doubles / floats per branch record (5 used, padded for alignment)
+template <typename T>
+__device__ __forceinline__ void gm_coef(const double* __restrict__ mc, double t, T* C) {
+    const double s = mc[0];
+    const double e1m = -expm1(-s * t);  // 1 - e^{-s t}
+    const double e1 = exp(-s * t);
+    C[0] = (T)e1m;
+#pragma unroll
+    for (int g = 0; g < 2; ++g) {
+        const double A = mc[1 + g], Pi = mc[3 + g];
+        const double eg = exp(-s * A * t);
+        // e^{-s t} - e^{-s A t} without cancellation
+        const double d = A >= 1.0 ? e1 * -expm1(-s * (A - 1.0) * t) : -eg * -expm1(-s * (1.0 - A) * t);
+        C[1 + g] = (T)(d / Pi);
+        C[3 + g] = (T)eg;
+    }
+#pragma unroll
+    for (int k = 5; k < GMC; ++k) C[k] = T(0);
+}
+template <typename T>
+__device__ __forceinline__ void gm_branch_c(T (&R)[4], const T* __restrict__ C, const T (&pi)[4]) {
+    const T gR = fma(pi[2], R[2], pi[0] * R[0]);
+    const T gY = fma(pi[3], R[3], pi[1] * R[1]);
+    const T aT = C[0] * (gR + gY);
+    const T xR = fma(C[1], gR, aT), xY = fma(C[2], gY, aT);
+    R[0] = fma(C[3], R[0], xR);
+    R[2] = fma(C[3], R[2], xR);
+    R[1] = fma(C[4], R[1], xY);
+    R[3] = fma(C[4], R[3], xY);
+}
+// column x of P(t) (the branch-transformed indicator of base x): P_{i x}
+template <typename T>
+__device__ __forceinline__ void gm_col_c(T (&v)[4], const T* __restrict__ C, int x, const T (&pi)[4]) {
+    const int gx = x & 1;
+#pragma unroll
+    for (int i = 0; i < 4; ++i) {
+        const int g = i & 1;
+        T p = C[0] * pi[x];
+        if (g == gx) p = fma(C[1 + g], pi[x], p);
+        if (i == x) p += C[3 + g];
+        v[i] = p;
+    }
+}
+
 template <typename T, int D, int S, bool AMB>
 __device__ __forceinline__ void gm_tt(T (&R)[D][4], uint32_t code, const T* __restrict__ P,
                                       const uint8_t* __restrict__ codes, int Lpad, int site, int& scale) {
@@ -563,7 +613,7 @@ struct UpBr {
         }
     }
     __device__ __forceinline__ void apply(T (&v)[4], const T (&pi)[4]) const {
-        if constexpr (GM) gm_branch<T>(v, e);
+        if constexpr (GM) gm_branch_c<T>(v, e, pi);  // e -> the structured branch record
         else branch<T>(v, e, em, pi);
     }
 };
@@ -728,7 +778,7 @@ template <typename T, int DR, int SI, bool PT, bool GM = false>
 __host__ __device__ size_t tab_smem_bytes(int nops, int need, int trip_cap) {
     const int n = nops + 1;
     const int spill = need > DR ? need - DR : 0;
-    return align16(GM ? 32 * sizeof(T) * nops + 16 * sizeof(T) : sizeof(typename Traits<T>::E4) * nops) +
+    return align16(GM ? 2 * GMC * sizeof(T) * nops + GMC * sizeof(T) : sizeof(typename Traits<T>::E4) * nops) +
            align16(sizeof(T) * ((PT ? 32 : 16) * (size_t)n + (size_t)TRIP_EXTRA * (PT ? trip_cap : 0))) +
            align16(sizeof(OpRec<T>) * nops) + 2 * align16(Codes<SI>::buf_bytes(n)) +
            sizeof(T) * (size_t)spill * SI * 4 * PRUNE_THREADS +
@@ -757,13 +807,13 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
     using CD = Codes<SI>;
     constexpr uint32_t TABE = PT ? 32u : 16u;  // table entries per tip
     constexpr int BATCH = CD::BATCH;  // sites per batch
-    constexpr size_t OPB = GM ? 32 * sizeof(T) : sizeof(E4);  // branch data bytes per op
+    constexpr size_t OPB = GM ? 2 * GMC * sizeof(T) : sizeof(E4);  // branch data bytes per op
     const int nops = a.nops, n = nops + 1;
     const int trip_cap = PT ? a.trip_cap : 0;
     E4* s_e = reinterpret_cast<E4*>(smem_raw);  // F81: {e_a, em_a, e_b, em_b} per op
-    T* s_P = reinterpret_cast<T*>(smem_raw);    // general model: {P_a, P_b} per op
-    // general model: {P_a, P_b} of every op, then the identity (the root's up branch)
-    T* s_tab = reinterpret_cast<T*>(smem_raw + align16(OPB * nops + (GM ? 16 * sizeof(T) : 0)));
+    T* s_P = reinterpret_cast<T*>(smem_raw);    // general model: branch records {C_a, C_b} per op
+    // general model: {C_a, C_b} of every op, then the identity record (the root's up branch)
+    T* s_tab = reinterpret_cast<T*>(smem_raw + align16(OPB * nops + (GM ? GMC * sizeof(T) : 0)));
     // compacted ops: {code, table byte offset, original op index, tip c of a fused triplet}
     OpRec<T>* s_opc = reinterpret_cast<OpRec<T>*>(reinterpret_cast<unsigned char*>(s_tab) +
                                             align16(sizeof(T) * (TABE * n + (size_t)TRIP_EXTRA * trip_cap)));
@@ -809,20 +859,21 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
             s_d[2 * i + 1] = Bounds<T>::ilogb((T)ed.w) + lp;
         }
     }
-    if constexpr (GM) {  // {P_a, P_b} of every op from its branch lengths {t_a, 0, t_b, 0}; d = min_XY P_XY(t)
+    if constexpr (GM) {  // {C_a, C_b} of every op from its branch lengths {t_a, 0, t_b, 0}; d = min_XY P_XY(t)
         for (int i = tid; i < nops * 2; i += PRUNE_THREADS) {
             const E4 ed = ge[i >> 1];
-            double P[16];
-            pmat(a.gm, (double)((i & 1) ? ed.z : ed.x), P);
-            T pmin = (T)P[0];
+            T* C = s_P + i * GMC;
+            gm_coef<T>(a.gm + 36, (double)((i & 1) ? ed.z : ed.x), C);
+            T pmin = T(1);
 #pragma unroll
-            for (int k = 0; k < 16; ++k) {
-                s_P[i * 16 + k] = (T)P[k];
-                pmin = min(pmin, (T)P[k]);
+            for (int x = 0; x < 4; ++x) {
+                T col[4];
+                gm_col_c<T>(col, C, x, pi);
+                pmin = min(pmin, min(min(col[0], col[1]), min(col[2], col[3])));
             }
             s_d[i] = Bounds<T>::ilogb(pmin);
         }
-        if (tid < 16) s_P[nops * 32 + tid] = (tid % 5 == 0) ? T(1) : T(0);  // identity: the root's up branch
+        if (tid < GMC) s_P[nops * 2 * GMC + tid] = (tid == 3 || tid == 4) ? T(1) : T(0);  // identity: a = b = 0, c = 1
     }
     __syncthreads();
     PTS(2);
@@ -890,7 +941,7 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
         const uint32_t xi = s_opc[i].h.x;
         const int ty = (int)(xi & 3u), sp = (int)((xi >> 2) & 15u);
         const int lvl = (ty == (int)OP_TS) ? sp - 1 : (ty == (int)OP_SS ? sp - 2 : sp);
-        T up0 = GM ? (T)(nops * 32) : T(1), up1 = T(0);
+        T up0 = GM ? (T)(nops * 2 * GMC) : T(1), up1 = T(0);
         for (int j = i + 1; j < nops_c; ++j) {
             const uint4 oj = s_opc[j].h;
             const int tj = (int)(oj.x & 3u), sj = (int)((oj.x >> 2) & 15u);
@@ -899,7 +950,7 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
                              : (tj == (int)OP_SS && sj - 1 == lvl) ? 1 : -1;
             if (side < 0) continue;
             if constexpr (GM) {
-                up0 = (T)(oj.z * 32u + (uint32_t)side * 16u);
+                up0 = (T)(oj.z * 2u * GMC + (uint32_t)side * GMC);
             } else {
                 const E4 e = s_e[oj.z];
                 up0 = side ? (T)e.z : (T)e.x;
@@ -933,33 +984,29 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
             tab = reinterpret_cast<T*>(reinterpret_cast<char*>(s_tab) + (ox.y & ~TAB_CHECK));
             T va[4], vb[4];
             if constexpr (GM) {  // tip vectors are columns of P (row X = parent state)
-                const T* Pa = s_P + ox.z * 32;
-                auto col = [](T (&w)[4], const T* P, int x) {
-#pragma unroll
-                    for (int X = 0; X < 4; ++X) w[X] = P[X * 4 + x];
-                };
+                const T* Ca = s_P + ox.z * 2 * GMC;
                 if (ty == OP_TT && PT) {
-                    col(va, Pa, r >> 2);
-                    col(vb, Pa + 16, r & 3);
+                    gm_col_c<T>(va, Ca, r >> 2, pi);
+                    gm_col_c<T>(vb, Ca + GMC, r & 3, pi);
 #pragma unroll
                     for (int X = 0; X < 4; ++X) v[0][X] = va[X] * vb[X];
                     tabop = true;
                 } else if (ty == OP_TT && r < 8) {
-                    col(va, Pa + (r < 4 ? 0 : 16), r & 3);
+                    gm_col_c<T>(va, Ca + (r < 4 ? 0 : GMC), r & 3, pi);
                     st4<T>(tab + r * 4, va);
                 } else if (ty == OP_TS && r < 4) {
-                    col(va, Pa, r);
+                    gm_col_c<T>(va, Ca, r, pi);
                     st4<T>(tab + r * 4, va);
-                } else if (ty == OP_TTT) {  // op o: P_a, P_b; op o+1: P of tip c, P of the cherry's branch
-                    const T* Pc = Pa + 32;
-                    col(va, Pa, r >> 2);
-                    col(vb, Pa + 16, r & 3);
+                } else if (ty == OP_TTT) {  // op o: C_a, C_b; op o+1: C of tip c, C of the cherry's branch
+                    const T* Cc = Ca + 2 * GMC;
+                    gm_col_c<T>(va, Ca, r >> 2, pi);
+                    gm_col_c<T>(vb, Ca + GMC, r & 3, pi);
 #pragma unroll
                     for (int X = 0; X < 4; ++X) va[X] *= vb[X];
-                    gm_branch<T>(va, Pc + 16);
+                    gm_branch_c<T>(va, Cc + GMC, pi);
 #pragma unroll
                     for (int xc = 0; xc < 4; ++xc) {
-                        col(vb, Pc, xc);
+                        gm_col_c<T>(vb, Cc, xc, pi);
 #pragma unroll
                         for (int X = 0; X < 4; ++X) v[xc][X] = vb[X] * va[X];
                     }
