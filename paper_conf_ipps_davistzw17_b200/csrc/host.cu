@@ -663,13 +663,13 @@ void upgma(int n, int L, const uint8_t* codes, double theta0, int32_t* parent, d
 #ifndef MPCGS_SETUP
 #define MPCGS_SETUP 3.0
 #endif
-void prune_tiling(int n, int L, int ntrees, int precision, int& tiles, int& sites_per_cta) {
+void prune_tiling(int n, int L, int ntrees, int precision, int& tiles, int& sites_per_cta, int model = 0) {
     const int batch = prune_batch_sites(n, precision);
     const int unit = prune_unit_batches(n, L, precision);
     const double trees = (double)std::max(ntrees, 1);
     const long batches = (L + batch - 1) / batch;
     const long units = (batches + unit - 1) / unit;
-    const double slots = 148.0 * (precision == 32 ? 4.0 : 3.0);  // resident CTAs (occupancy of the table kernel)
+    const double slots = 148.0 * prune_resident_per_sm(n, precision, model != 0);  // resident CTAs
     const long tmin = std::max<long>(1, (units * unit + MPCGS_MAXPER - 1) / MPCGS_MAXPER);
     double best = 1e300;
     long bt = tmin;
@@ -719,7 +719,7 @@ PruneArgs prune_args(mpcgs_ctx* c, int ntrees, double* out, int out_first, int o
     a.gm = c->model ? c->s.gm : nullptr;
     a.amb = c->s.amb;
     a.sched_P = c->s.sched_P;
-    prune_tiling(c->n, c->L, ntrees, c->precision, a.tiles, a.sites_per_cta);
+    prune_tiling(c->n, c->L, ntrees, c->precision, a.tiles, a.sites_per_cta, c->model);
     a.unit_batches = prune_unit_batches(c->n, c->L, c->precision);
     a.unit_sites = a.unit_batches * prune_batch_sites(c->n, c->precision);
     a.units = (c->L + a.unit_sites - 1) / a.unit_sites;

@@ -61,6 +61,7 @@ int prune_max_need(int n);
 int prune_need_cap(int n);
 int prune_batch_sites(int n, int precision);  // sites_per_cta must be a multiple of this
 bool prune_uses_tables(int n, int precision, bool general_model = false);
+int prune_resident_per_sm(int n, int precision, bool general_model = false);  // tiling cost model
 cudaError_t launch_prune(const PruneArgs& a, int ntrees, int depth, int precision, cudaStream_t st,
                          int* n_launched = nullptr);
 

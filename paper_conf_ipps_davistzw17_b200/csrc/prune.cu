@@ -23,7 +23,7 @@ int prune_max_need(int n) {
 // sites interleaved per thread: 4 for n <= 128 (product tables), 2 for larger
 // trees, whose codes / tables / spill levels take more shared memory
 static int prune_si(int n, int precision) {
-    if (!product_tables(n)) return 2;
+    if (!wide_sites(n)) return 2;
     return precision == 32 ? PRUNE_SI32 : PRUNE_SI64;
 }
 int prune_batch_sites(int n, int precision) { return PRUNE_THREADS * prune_si(n, precision); }
@@ -54,13 +54,25 @@ template <typename T, bool GM>
 static size_t tab_bytes_for(int n) {
     const int cap = prune_need_cap(n);
     constexpr int SI = sizeof(T) == 4 ? PRUNE_SI32 : PRUNE_SI64;
-    return product_tables(n) ? tab_smem_bytes<T, PRUNE_DR, SI, true, GM>(n - 1, cap, 0)
+    const bool pt = product_tables<T, GM>(n);
+    if (pt && !wide_sites(n)) return tab_smem_bytes<T, PRUNE_DR, PRUNE_SI_LARGE, true, GM>(n - 1, cap, 0);
+    return pt ? tab_smem_bytes<T, PRUNE_DR, SI, true, GM>(n - 1, cap, 0)
                              : tab_smem_bytes<T, PRUNE_DR, PRUNE_SI_LARGE, false, GM>(n - 1, cap, 0);
 }
 
 #ifndef MPCGS_TAB_MIN_N
 #define MPCGS_TAB_MIN_N 8  // below 8 tips the table setup costs more than it saves (c1: 41 -> 37 us per step)
 #endif
+// resident table-kernel CTAs per SM for the tiling cost model: the register limit
+// (159 registers FP64 -> 3, FP32 -> 4) or the shared-memory limit of the base layout
+int prune_resident_per_sm(int n, int precision, bool general_model) {
+    size_t bytes;
+    if (precision == 32) bytes = general_model ? tab_bytes_for<float, true>(n) : tab_bytes_for<float, false>(n);
+    else bytes = general_model ? tab_bytes_for<double, true>(n) : tab_bytes_for<double, false>(n);
+    const int by_smem = (int)((228 * 1024) / (bytes + 1024 + 256));
+    return std::max(1, std::min(precision == 32 ? 4 : 3, by_smem));
+}
+
 bool prune_uses_tables(int n, int precision, bool general_model) {
     if (n < MPCGS_TAB_MIN_N) return false;
     size_t bytes;

@@ -1283,8 +1283,22 @@ static cudaError_t launch_tab(const PruneArgs& a, int ntrees, cudaStream_t st) {
                     : launch_tab_w<T, DR, SI, PT, DMX, false, GM>(a, ntrees, st);
 }
 
-inline bool product_tables(int n) { return n <= 128; }  // 16x4 cherry tables (and SI sites/thread)
 constexpr int PRUNE_SI_LARGE = 2;  // sites per thread for n > 128
+inline bool wide_sites(int n) { return n <= 128; }  // SI sites per thread (else PRUNE_SI_LARGE)
+// cherry (16x4) / fused-triplet (64x4) tables: always up to 128 tips; above (with 2 sites
+// per thread) only while their shared memory still leaves two CTAs per SM (measured:
+// FP64 n = 192 +12 %, FP32 n = 256 +43 %; FP64 n = 256 needs one CTA per SM and is 20 %
+// slower with tables than without)
+#ifndef MPCGS_PT_SMEM_MAX
+#define MPCGS_PT_SMEM_MAX (110 * 1024)
+#endif
+template <typename T, bool GM>
+inline bool product_tables(int n) {
+    if (n <= 128) return true;
+    if (n > 256) return false;
+    return tab_smem_bytes<T, PRUNE_DR, PRUNE_SI_LARGE, true, GM>(n - 1, std::min(8, PRUNE_DR + PRUNE_SPILL), 0) <=
+           (size_t)MPCGS_PT_SMEM_MAX;
+}
 
 template <typename T, int SI, bool PT, bool GM>
 static cudaError_t launch_tab_dmx(const PruneArgs& a, int ntrees, cudaStream_t st) {
@@ -1332,7 +1346,9 @@ cudaError_t launch_prune_typed(PruneArgs a, int ntrees, int depth, cudaStream_t 
     a.need_cap = prune_need_cap(n);
     const bool deep = prune_max_need(n) > a.need_cap && a.tree_need != nullptr;
     if (!deep) a.tree_need = nullptr;
-    cudaError_t e = product_tables(n) ? launch_tab_dmx<T, SI, true, GM>(a, ntrees, st)
+    const bool pt = product_tables<T, GM>(n);
+    cudaError_t e = (pt && !wide_sites(n)) ? launch_tab_dmx<T, PRUNE_SI_LARGE, true, GM>(a, ntrees, st)
+                    : pt ? launch_tab_dmx<T, SI, true, GM>(a, ntrees, st)
                                       : launch_tab_dmx<T, PRUNE_SI_LARGE, false, GM>(a, ntrees, st);
     nl += 1;
     if (e != cudaSuccess || !deep) return e;
