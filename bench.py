@@ -424,6 +424,29 @@ def main():
     if dist is not None:
         dist.all_reduce(t, op=dist.ReduceOp.MAX)
     loop_ms, prune_ms, propose_ms, draw_ms = (float(x) for x in t)
+    # the production loop as a user runs it (CUDA graphs of 32 steps, no per-phase events,
+    # no L2 flush: steady state with a warm L2), CUDA events on the caller's stream; short
+    # steps run 256 of them so that the per-call graph capture is amortised as in real use
+    ctx.mpcgs_set_timing(0)
+    prod_steps = args.steps if loop_ms / args.steps > 1.0 else max(args.steps, 256)  # loop_ms: max over ranks
+    ctxp = ctx if prod_steps == args.steps else P.Context(
+        rows, wl["theta0"], precision=args.precision, max_proposals=N, max_samples=N * prod_steps,
+        init_tree=(wl["true_parent"], wl["true_age"]), rank=rank, world=world, nccl_id=fresh_nccl_id(),
+        stream=stream, incremental=args.incremental, compress_patterns=args.compress, model=args.model,
+        kappa=args.kappa, ambiguity=args.ambiguity > 0)
+    ctxp.mpcgs_sample(N, N * min(32, prod_steps), wl["chain_seed"] + 3)  # warm
+    barrier()
+    pe0, pe1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    pe0.record()
+    ctxp.mpcgs_sample(N, N * prod_steps, wl["chain_seed"] + 2)
+    pe1.record()
+    barrier()
+    tp = torch.tensor([pe0.elapsed_time(pe1)], dtype=torch.float64, device="cuda")
+    if dist is not None:
+        dist.all_reduce(tp, op=dist.ReduceOp.MAX)
+    prod_ms = float(tp[0]) * args.steps / prod_steps  # per args.steps steps
+    if ctxp is not ctx:
+        ctxp.free()
     partials = N * L * (n - 1) * args.steps
     value = partials / (loop_ms / 1e3)
     ms_per_step = loop_ms / args.steps
@@ -568,6 +591,11 @@ def main():
             "vs_baseline": None, "dtype": "f64" if args.precision == 64 else "f32", "data": "synthetic",
             "config": workload_config(args, wl), "proposals_per_s": N * args.steps / (loop_ms / 1e3),
             "roofline": roof, "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": int(launches),
+            "production_loop": {"ms_per_step": prod_ms / args.steps, "value": partials / (prod_ms / 1e3),
+                                "steps": prod_steps,
+                                "note": "mpcgs_sample as shipped (CUDA graphs, no per-phase events, L2 not "
+                                        "flushed: warm-L2 steady state); the headline value flushes L2 "
+                                        "between steps as the benchmark contract asks"},
             "phases_ms_per_step": {"context+propose": propose_ms / args.steps, "prune": prune_ms / args.steps,
                                    "exchange+draw+commit": draw_ms / args.steps,
                                    "source": "CUDA events around each phase of every timed step "

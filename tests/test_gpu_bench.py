@@ -23,7 +23,7 @@ def test_bench_line_contract():
     d = _run("--workload", "c2", "--steps", "4", "--warmup", "3", "--cpu-seconds", "2")
     for k in ("metric", "value", "unit", "n_gpus", "steps", "warmup", "ms_per_step", "higher_is_better", "dtype",
               "config", "roofline", "cpu_baseline", "e2e", "gpu_launches", "clocks", "theta_mle",
-              "phases_ms_per_step"):
+              "phases_ms_per_step", "production_loop"):
         assert k in d, k
     assert d["value"] > 0 and d["gpu_launches"] > 0
     r = d["roofline"]
