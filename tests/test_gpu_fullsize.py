@@ -31,8 +31,11 @@ CASES = [
 ]
 
 
+@pytest.mark.parametrize("precision,incremental", [(64, False), (32, False), (64, True)])
 @pytest.mark.parametrize("name,over,n_ll", CASES)
-def test_full_size_step_sampled_parity(P, orc, name, over, n_ll):
+def test_full_size_step_sampled_parity(P, orc, name, over, n_ll, precision, incremental):
+    if (precision, incremental) != (64, False) and name != "c5":
+        pytest.skip("FP32 and incremental rescoring are checked at the bench workload")
     wl = synth.workload(name, **over)
     codes = wl["codes"]
     n, L = codes.shape
@@ -41,7 +44,9 @@ def test_full_size_step_sampled_parity(P, orc, name, over, n_ll):
     u = orc.default_rate(pi)
     theta0 = wl["theta0"]
     parent, age = wl["true_parent"], wl["true_age"]
-    ctx = P.Context(synth.to_strings(codes), theta0, init_tree=(parent, age), max_proposals=N, max_samples=16)
+    ctx = P.Context(synth.to_strings(codes), theta0, init_tree=(parent, age), max_proposals=N, max_samples=16,
+                    precision=precision, incremental=incremental)
+    tol = 1e-9 if precision == 64 else 1e-4
     seed, step = wl["chain_seed"], 3
     tr = ctx.mpcgs_step_trace(step, N, N, seed)
     assert tr["target"] == orc.pick_target(parent, seed, step)
@@ -59,8 +64,10 @@ def test_full_size_step_sampled_parity(P, orc, name, over, n_ll):
         assert abs(tr["S"][slot] - orc.coalescent_S(a2, n)) <= 1e-12 * abs(tr["S"][slot])
         if slot in ll_slots:
             want = orc.log_likelihood(codes, p2, a2, pi, u)
-            assert abs(tr["logL"][slot] - want) <= 1e-9 * abs(want), (slot, tr["logL"][slot], want)
+            assert abs(tr["logL"][slot] - want) <= tol * abs(want), (slot, tr["logL"][slot], want)
     assert flagged <= 2
+    if precision == 32:  # FP32 gets logL tolerance, not index parity (P21)
+        return
     # draws: inverse CDF over softmax of the GPU likelihoods, lowest index on ties
     w, cum = orc.weights(tr["logL"])
     for d, got in enumerate(tr["draws"]):

@@ -400,3 +400,16 @@ def test_init_newick_equals_arrays(P, orc):
     with pytest.raises(P.MpcgsError) as ei:
         _ctx(P, codes, wl["theta0"], init_newick="((0:1,1:1):1,2:2);", max_proposals=8, max_samples=8)
     assert ei.value.status == -1 and "init_newick" in str(ei.value)
+
+
+def test_all_weights_non_finite_is_numeric_error(P):
+    """S6 / MPCGS_E_NUMERIC: a user pi with pi_T = 0 on data containing T makes every
+    genealogy's likelihood 0 (the root sum weights state T by pi_T), so all N + 1 weights
+    are non-finite: mpcgs_sample reports MPCGS_E_NUMERIC instead of drawing."""
+    rows = ["ACGTACGTAC", "ACGAACGTAC", "ACGTACGAAC", "TCGAACGTAC"]
+    ctx = P.Context(rows, 0.1, base_freq=[0.4, 0.3, 0.3, 0.0], mu=1.0, max_proposals=8, max_samples=16)
+    _, _, gl, _ = ctx.mpcgs_get_state()
+    assert gl == -np.inf
+    with pytest.raises(P.MpcgsError) as ei:
+        ctx.mpcgs_sample(8, 16, 1)
+    assert ei.value.status == -7
