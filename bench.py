@@ -266,7 +266,7 @@ def workload_config(args, wl):
                else ""),
             "model": args.model + ("" if args.model == "F81" else f" (kappa {args.kappa}; SURVEY 8(f) f4)"),
             "ambiguity": (f"{args.ambiguity:g} of characters IUPAC ambiguity codes + {args.ambiguity / 2:g} N "
-                          "(SURVEY 8(f) f4; flat kernel)" if args.ambiguity > 0 else "none")}
+                          "(SURVEY 8(f) f4; 4-bit base-set tables)" if args.ambiguity > 0 else "none")}
 
 
 def run_loci(args, over):
@@ -471,7 +471,7 @@ def main():
             "lds_peak_measured_gbs": alu["lds_gbs"],
             "pipe": pipe_from_profiles(tag),
             "traffic": traffic_from_profiles(tag),
-            "kernel": ("k_prune (flat, base-set tips)" if args.ambiguity > 0 else "k_prune_tab")
+            "kernel": ("k_prune_tab (4-bit base-set tip codes)" if args.ambiguity > 0 else "k_prune_tab")
                       + (" + general model (F84/HKY85)" if gm else ""),
             "prune_share_of_step": prune_ms / loop_ms,
             "partials_per_s_prune_only": N * L * (n - 1) / (prune_avg_s * world) if world == 1 else
@@ -567,7 +567,8 @@ def main():
         Mm = 1_000_000
         rng = np.random.default_rng(17)
         S_m = rng.gamma(n - 1, 0.012, Mm) * np.exp(rng.normal(0.0, 0.2, Mm))
-        ctx4 = P.Context(rows[:min(n, 64)], wl["theta0"], max_proposals=1, max_samples=Mm, stream=stream)
+        ctx4 = P.Context(rows[:min(n, 64)], wl["theta0"], max_proposals=1, max_samples=Mm, stream=stream,
+                         ambiguity=args.ambiguity > 0)
         ctx4.mpcgs_load_samples(S_m, wl["theta0"])
         ctx4.mpcgs_estimate_theta(256)
         best = 1e30

@@ -156,7 +156,7 @@ Layout layout(int n, int L, int Nmax, int64_t Mmax, int precision, int increment
         return r;
     };
     y.codes = take((size_t)n * Lpad);
-    y.codes2 = take(4 * (size_t)n * codes2_words(L));
+    y.codes2 = take(8 * (size_t)n * codes2_words(L));  // room for 4-bit base-set codes (ambiguity data)
     y.parent = take(4 * (size_t)nn);
     y.left = take(4 * (size_t)nn);
     y.right = take(4 * (size_t)nn);
@@ -709,7 +709,7 @@ PruneArgs prune_args(mpcgs_ctx* c, int ntrees, double* out, int out_first, int o
     a.codes = c->s.codes;
     a.codes2 = c->codes2;
     a.site_w = c->s.site_w;
-    a.W2 = codes2_words(c->L);
+    a.W2 = codes2_words(c->L) * (c->s.amb ? 2 : 1);  // 4-bit codes with ambiguity data
     a.Lpad = c->Lpad;
     a.L = c->L;
     a.nops = c->nops;
@@ -1303,7 +1303,7 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
         s.Mmax = c->Mmax;
         c->theta_cnt = (unsigned*)(b + y.theta_cnt);
         c->score_out = (double*)(b + y.score_out);
-        c->codes2 = any_amb ? nullptr : (uint32_t*)(b + y.codes2);  // 2-bit codes: unambiguous data only
+        c->codes2 = (uint32_t*)(b + y.codes2);  // 2-bit base codes, or 4-bit base-set masks (ambiguity data)
         s.amb = any_amb ? 1 : 0;
         s.site_w = cfg->compress_patterns ? (const double*)(b + y.site_w) : nullptr;
         if ((st = enter(c))) break;
@@ -1312,16 +1312,23 @@ mpcgs_status mpcgs_init(const mpcgs_alignment* aln, const mpcgs_config* cfg, dou
         // byte codes (the flat kernel) are unpacked on the device from the 2-bit words
         // unless the data hold ambiguity codes (then they are the only codes)
         std::vector<uint8_t> padded(any_amb ? (size_t)n * c->Lpad : 0, 0);
-        const int W2 = codes2_words(L);
+        const int W2 = codes2_words(L), W4 = 2 * W2;
         const int si2 = prune_batch_sites(n, c->precision) / PRUNE_THREADS;  // sites per thread of the table kernel
-        std::vector<uint32_t> packed((size_t)n * W2, 0u);
-        int shift[16];  // thread-interleaved order of the table kernel (Codes): site k of thread q
+        std::vector<uint32_t> packed((size_t)n * (any_amb ? W4 : W2), 0u);
+        // thread-interleaved order of the table kernel (Codes<SI, BITS>): site k of thread q
+        int shift[16], shift4[8];
         for (int s16 = 0; s16 < 16; ++s16) shift[s16] = (32 / si2) * (s16 % si2) + 2 * (s16 / si2);
+        for (int s8 = 0; s8 < 8; ++s8) shift4[s8] = (32 / si2) * (s8 % si2) + 4 * (s8 / si2);
         parallel_rows(n, [&](int i) {
             const uint8_t* src = codes.data() + (size_t)i * L;
-            if (any_amb) {  // byte codes: base-set masks 1..15
+            if (any_amb) {  // byte codes and 4-bit codes: base-set masks 1..15
                 uint8_t* pb = padded.data() + (size_t)i * c->Lpad;
-                for (int site = 0; site < L; ++site) pb[site] = (uint8_t)base_set(src[site]);
+                uint32_t* pw = packed.data() + (size_t)i * W4;
+                for (int site = 0; site < L; ++site) {
+                    const uint32_t m = (uint32_t)base_set(src[site]);
+                    pb[site] = (uint8_t)m;
+                    pw[site >> 3] |= m << shift4[site & 7];
+                }
                 return;
             }
             uint32_t* pw = packed.data() + (size_t)i * W2;

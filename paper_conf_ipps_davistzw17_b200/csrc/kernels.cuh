@@ -30,7 +30,7 @@ struct PruneArgs {
     const void* sched_e;       // [ntrees][nops] float4 / double4
     const double* gm;          // general model (f4): [36] eigen-system of Q, else nullptr (F81)
     void* sched_P;             // general model: [ntrees][nops][32] P matrices (float / double)
-    int amb;                   // byte codes are base-set masks (ambiguity codes): flat kernel only
+    int amb;                   // base-set codes (ambiguity, S24): byte masks (flat kernel), 4-bit codes2 (tables)
     // site tiles: tile t covers exact-sum units [t*units/tiles, (t+1)*units/tiles) of
     // unit_sites sites each (balanced; tile_range below); sites_per_cta = the largest tile
     int tiles, sites_per_cta, units, unit_sites;
@@ -60,7 +60,7 @@ int prune_depth_for(int n);
 int prune_max_need(int n);
 int prune_need_cap(int n);
 int prune_batch_sites(int n, int precision);  // sites_per_cta must be a multiple of this
-bool prune_uses_tables(int n, int precision, bool general_model = false);
+bool prune_uses_tables(int n, int precision, bool general_model = false, bool amb = false);
 int prune_resident_per_sm(int n, int precision, bool general_model = false);  // tiling cost model
 cudaError_t launch_prune(const PruneArgs& a, int ntrees, int depth, int precision, cudaStream_t st,
                          int* n_launched = nullptr);

@@ -51,9 +51,12 @@ int prune_need_cap(int n) { return std::min(prune_max_need(n), PRUNE_DR + (n <= 
 
 
 template <typename T, bool GM>
-static size_t tab_bytes_for(int n) {
+static size_t tab_bytes_for(int n, bool amb = false) {
     const int cap = prune_need_cap(n);
     constexpr int SI = sizeof(T) == 4 ? PRUNE_SI32 : PRUNE_SI64;
+    if (amb)  // 4-bit base-set codes, 16-row tip tables (S24)
+        return wide_sites(n) ? tab_smem_bytes<T, PRUNE_DR, SI, false, GM, 4>(n - 1, cap, 0)
+                             : tab_smem_bytes<T, PRUNE_DR, PRUNE_SI_LARGE, false, GM, 4>(n - 1, cap, 0);
     const bool pt = product_tables<T, GM>(n);
     if (pt && !wide_sites(n)) return tab_smem_bytes<T, PRUNE_DR, PRUNE_SI_LARGE, true, GM>(n - 1, cap, 0);
     return pt ? tab_smem_bytes<T, PRUNE_DR, SI, true, GM>(n - 1, cap, 0)
@@ -73,11 +76,11 @@ int prune_resident_per_sm(int n, int precision, bool general_model) {
     return std::max(1, std::min(precision == 32 ? 4 : 3, by_smem));
 }
 
-bool prune_uses_tables(int n, int precision, bool general_model) {
+bool prune_uses_tables(int n, int precision, bool general_model, bool amb) {
     if (n < MPCGS_TAB_MIN_N) return false;
     size_t bytes;
-    if (precision == 32) bytes = general_model ? tab_bytes_for<float, true>(n) : tab_bytes_for<float, false>(n);
-    else bytes = general_model ? tab_bytes_for<double, true>(n) : tab_bytes_for<double, false>(n);
+    if (precision == 32) bytes = general_model ? tab_bytes_for<float, true>(n, amb) : tab_bytes_for<float, false>(n, amb);
+    else bytes = general_model ? tab_bytes_for<double, true>(n, amb) : tab_bytes_for<double, false>(n, amb);
     return bytes <= 160 * 1024;
 }
 

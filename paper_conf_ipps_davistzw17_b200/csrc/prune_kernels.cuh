@@ -444,17 +444,21 @@ struct Stack {
 // codes as bytes (SI = 4: bytes 0..3; SI = 2: bytes 0 and 2), so the entry index
 // of a cherry (4 a + b) or a fused triplet (16 a + 4 b + c) is formed for all SI
 // sites at once with byte-lane arithmetic (no carries: every lane stays < 64).
-template <int SI>
+// BITS = 4 (ambiguity codes): 4-bit base-set masks, 8 sites per
+// word, site k of thread q at bit (32/SI) k + 4 q; the lanes are then 0..15.
+template <int SI, int BITS = 2>
 struct Codes {
     uint32_t sbase;             // this batch's buffer (shared-window address)
     int wofs;                   // word index of this thread's sites
-    uint32_t qs;                // 2 q: this thread's bit offset in its word
+    uint32_t qs;                // BITS q: this thread's bit offset in its word
     static constexpr int BATCH = PRUNE_THREADS * SI;
-    static constexpr int WB = BATCH / 16;
-    static constexpr uint32_t MASK = SI == 4 ? 0x03030303u : 0x00030003u;
+    static constexpr int SPW = 32 / BITS;          // sites per word
+    static constexpr int WB = BATCH / SPW;         // words per tip row of a batch
+    static constexpr uint32_t LM = (1u << BITS) - 1u;
+    static constexpr uint32_t MASK = SI == 4 ? LM * 0x01010101u : LM * 0x00010001u;
     __device__ __forceinline__ void init(int tid) {
-        wofs = (tid * SI) >> 4;
-        qs = 2u * (uint32_t)(tid % (16 / SI));
+        wofs = (tid * SI) / SPW;
+        qs = (uint32_t)BITS * (uint32_t)(tid % (SPW / SI));
     }
     __device__ __forceinline__ uint32_t word(int tip) const {
         return lds_u32(sbase + (uint32_t)(tip * WB + wofs) * 4u);
@@ -618,9 +622,9 @@ struct UpBr {
     }
 };
 
-template <typename T, int DR, int SI, bool PT, int S, int DMX, bool GM>
+template <typename T, int DR, int SI, bool PT, int S, int DMX, bool GM, typename CD>
 __device__ __forceinline__ void tab_tt(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, uint32_t wa,
-                                       const UpBr<T, GM>& ub, uint32_t s_tab, const Codes<SI>& c,
+                                       const UpBr<T, GM>& ub, uint32_t s_tab, const CD& c,
                                        const T (&pi)[4], int (&scale)[SI]) {
     if constexpr (S < DMX) {
         constexpr int EB = 4 * sizeof(T);
@@ -642,7 +646,7 @@ __device__ __forceinline__ void tab_tt(Stack<T, DR, SI>& st, uint32_t code, uint
             for (int k = 0; k < SI; ++k) {
                 T w[4];
                 lds4(v[k], base + c.template off<EB>(la, k));
-                lds4(w, base + 16 * (uint32_t)sizeof(T) + c.template off<EB>(lb, k));
+                lds4(w, base + 4u * (CD::LM + 1u) * (uint32_t)sizeof(T) + c.template off<EB>(lb, k));  // table b after a
 #pragma unroll
                 for (int i = 0; i < 4; ++i) v[k][i] *= w[i];
             }
@@ -659,9 +663,9 @@ __device__ __forceinline__ void tab_tt(Stack<T, DR, SI>& st, uint32_t code, uint
 }
 
 // fused triplet: one lookup in the 64x4 table of branch_up(tip(c) (.) branch(tip(a) (.) tip(b)))
-template <typename T, int DR, int SI, bool PT, int S, int DMX, bool GM>
+template <typename T, int DR, int SI, bool PT, int S, int DMX, bool GM, typename CD>
 __device__ __forceinline__ void tab_ttt(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, uint32_t tc,
-                                        uint32_t wa, const UpBr<T, GM>& ub, uint32_t s_tab, const Codes<SI>& c,
+                                        uint32_t wa, const UpBr<T, GM>& ub, uint32_t s_tab, const CD& c,
                                         const T (&pi)[4], int (&scale)[SI]) {
     if constexpr (PT && S < DMX) {
         constexpr int EB = 4 * sizeof(T);
@@ -689,9 +693,9 @@ __device__ __forceinline__ void tab_ttt(Stack<T, DR, SI>& st, uint32_t code, uin
 // Fused (OP_FUSED kind 1 / 2): a cherry / triplet table op and the SS that merges
 // its result into the stack top, v = top (.) table(x_a, x_b[, x_c]) -- the table
 // already carries the cherry's branch into the SS, the op record the SS's up branch.
-template <typename T, int DR, int SI, int S, int DMX, bool GM>
+template <typename T, int DR, int SI, int S, int DMX, bool GM, typename CD>
 __device__ __forceinline__ void tab_ts(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, uint32_t tc,
-                                       uint32_t wa, const UpBr<T, GM>& ub, uint32_t s_tab, const Codes<SI>& c,
+                                       uint32_t wa, const UpBr<T, GM>& ub, uint32_t s_tab, const CD& c,
                                        const T (&pi)[4], int (&scale)[SI]) {
     if constexpr (S >= 1 && S <= DMX) {
         constexpr int EB = 4 * sizeof(T);
@@ -745,19 +749,19 @@ __device__ __forceinline__ void tab_ss(Stack<T, DR, SI>& st, uint32_t code, cons
 }
 
 #define MPCGS_TABCASE(S)                                                                          \
-    case 4 * (S) + 0: tab_tt<T, DR, SI, PT, S, DMX, GM>(st, code, toff, wa, ub, s_tab, cc, pi, scale); break;       \
-    case 4 * (S) + 1: tab_ts<T, DR, SI, S, DMX, GM>(st, code, toff, tc, wa, ub, s_tab, cc, pi, scale); break; \
+    case 4 * (S) + 0: tab_tt<T, DR, SI, PT, S, DMX, GM, CD>(st, code, toff, wa, ub, s_tab, cc, pi, scale); break;       \
+    case 4 * (S) + 1: tab_ts<T, DR, SI, S, DMX, GM, CD>(st, code, toff, tc, wa, ub, s_tab, cc, pi, scale); break; \
     case 4 * (S) + 2: tab_ss<T, DR, SI, S, DMX, GM>(st, code, ub, pi, scale); break;                      \
-    case 4 * (S) + 3: tab_ttt<T, DR, SI, PT, S, DMX, GM>(st, code, toff, tc, wa, ub, s_tab, cc, pi, scale); break;
+    case 4 * (S) + 3: tab_ttt<T, DR, SI, PT, S, DMX, GM, CD>(st, code, toff, tc, wa, ub, s_tab, cc, pi, scale); break;
 #define MPCGS_CASES_4 MPCGS_TABCASE(0) MPCGS_TABCASE(1) MPCGS_TABCASE(2) MPCGS_TABCASE(3) MPCGS_TABCASE(4)
 #define MPCGS_CASES_6 MPCGS_CASES_4 MPCGS_TABCASE(5) MPCGS_TABCASE(6)
 #define MPCGS_CASES_8 MPCGS_CASES_6 MPCGS_TABCASE(7) MPCGS_TABCASE(8)
 #define MPCGS_CASES_10 MPCGS_CASES_8 MPCGS_TABCASE(9) MPCGS_TABCASE(10)
 
 // one op for SI sites; the switch only has the (sp, type) labels a DMX-level tree can use
-template <typename T, int DR, int SI, bool PT, int DMX, bool GM>
+template <typename T, int DR, int SI, bool PT, int DMX, bool GM, typename CD>
 __device__ __forceinline__ void run_op(int di, Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, uint32_t tc,
-                                       uint32_t wa, const UpBr<T, GM>& ub, uint32_t s_tab, const Codes<SI>& cc,
+                                       uint32_t wa, const UpBr<T, GM>& ub, uint32_t s_tab, const CD& cc,
                                        const T (&pi)[4], int (&scale)[SI]) {
     if constexpr (DMX <= 4) {
         switch (di) { MPCGS_CASES_4 default: __builtin_unreachable(); }
@@ -774,13 +778,13 @@ __host__ __device__ constexpr size_t align16(size_t x) { return (x + 15) & ~(siz
 
 // shared memory of the table kernel for trees of n tips whose register need is
 // at most `need` (spill levels above DR), with up to `trip_cap` fused triplets
-template <typename T, int DR, int SI, bool PT, bool GM = false>
+template <typename T, int DR, int SI, bool PT, bool GM = false, int BITS = 2>
 __host__ __device__ size_t tab_smem_bytes(int nops, int need, int trip_cap) {
     const int n = nops + 1;
     const int spill = need > DR ? need - DR : 0;
     return align16(GM ? 2 * GMC * sizeof(T) * nops + GMC * sizeof(T) : sizeof(typename Traits<T>::E4) * nops) +
-           align16(sizeof(T) * ((PT ? 32 : 16) * (size_t)n + (size_t)TRIP_EXTRA * (PT ? trip_cap : 0))) +
-           align16(sizeof(OpRec<T>) * nops) + 2 * align16(Codes<SI>::buf_bytes(n)) +
+           align16(sizeof(T) * ((PT ? 32 : (BITS == 4 ? 64 : 16)) * (size_t)n + (size_t)TRIP_EXTRA * (PT ? trip_cap : 0))) +
+           align16(sizeof(OpRec<T>) * nops) + 2 * align16(Codes<SI, BITS>::buf_bytes(n)) +
            sizeof(T) * (size_t)spill * SI * 4 * PRUNE_THREADS +
            align16(sizeof(int) * 2 * (size_t)nops) + align16(sizeof(int) * (size_t)nops) + 64 * sizeof(int);
 }
@@ -800,12 +804,13 @@ static __device__ long long g_pts[8];
 // One CTA scores genealogy `tree` over site tile `tile`; its schedule is gop / ge
 // (global memory written by k_propose); smem_raw = the
 // dynamic shared memory of tab_smem_bytes.
-template <typename T, int DR, int SI, bool PT, int DMX, bool W, bool GM>
+template <typename T, int DR, int SI, bool PT, int DMX, bool W, bool GM, int BITS>
 __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int tile, const uint32_t* gop,
                                                const typename Traits<T>::E4* ge, unsigned char* smem_raw) {
     using E4 = typename Traits<T>::E4;
-    using CD = Codes<SI>;
-    constexpr uint32_t TABE = PT ? 32u : 16u;  // table entries per tip
+    using CD = Codes<SI, BITS>;
+    static_assert(BITS == 2 || !PT, "4-bit (ambiguity) codes use tip tables only");
+    constexpr uint32_t TABE = PT ? 32u : (BITS == 4 ? 64u : 16u);  // table values per tip
     constexpr int BATCH = CD::BATCH;  // sites per batch
     constexpr size_t OPB = GM ? 2 * GMC * sizeof(T) : sizeof(E4);  // branch data bytes per op
     const int nops = a.nops, n = nops + 1;
@@ -836,7 +841,7 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
         const int site0 = s_begin + b * BATCH;
         unsigned char* dst = s_cod + (size_t)buf * bufb;
         constexpr int WB = CD::WB, CH = WB / 4;  // 16-byte chunks per tip row
-        const uint32_t* src = a.codes2 + (site0 >> 4);
+        const uint32_t* src = a.codes2 + site0 / CD::SPW;
         for (int c = tid; c < n * CH; c += PRUNE_THREADS) {
             const int tip = c / CH, q = c - tip * CH;
             cp_async16(dst + ((size_t)tip * WB + q * 4) * 4, src + (size_t)tip * a.W2 + q * 4);
@@ -899,7 +904,7 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
             const bool prev = tid == 0 ? prev_start != 0u : ((ms >> (tid - 1)) & 1u) != 0u;
             const bool keep = i < nops && !(ty == OP_TS && prev);
             uint32_t sz = 0;
-            if (keep) sz = start ? 256u : (ty == OP_TT ? 2u * TABE : (ty == OP_TS ? 16u : 0u));
+            if (keep) sz = start ? 256u : (ty == OP_TT ? 2u * TABE : (ty == OP_TS ? (BITS == 4 ? 64u : 16u) : 0u));
             const unsigned mk = __ballot_sync(0xffffffffu, keep);
             const uint32_t j = c_keep + __popc(mk & ((1u << tid) - 1u));
             uint32_t x = sz;
@@ -991,6 +996,25 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
 #pragma unroll
                     for (int X = 0; X < 4; ++X) v[0][X] = va[X] * vb[X];
                     tabop = true;
+                } else if (BITS == 4 && (ty == OP_TT || ty == OP_TS)) {  // 16-row base-set tables (S24)
+                    auto setcol = [&](T (&w)[4], const T* C, int m) {
+#pragma unroll
+                        for (int X = 0; X < 4; ++X) w[X] = T(0);
+#pragma unroll
+                        for (int x = 0; x < 4; ++x)
+                            if ((m >> x) & 1) {
+                                T col[4];
+                                gm_col_c<T>(col, C, x, pi);
+#pragma unroll
+                                for (int X = 0; X < 4; ++X) w[X] += col[X];
+                            }
+                    };
+                    setcol(va, Ca, r);
+                    st4<T>(tab + r * 4, va);
+                    if (ty == OP_TT) {  // table b after table a
+                        setcol(vb, Ca + GMC, r);
+                        st4<T>(tab + (16 + r) * 4, vb);
+                    }
                 } else if (ty == OP_TT && r < 8) {
                     gm_col_c<T>(va, Ca + (r < 4 ? 0 : GMC), r & 3, pi);
                     st4<T>(tab + r * 4, va);
@@ -1021,6 +1045,13 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
 #pragma unroll
                     for (int X = 0; X < 4; ++X) v[0][X] = va[X] * vb[X];
                     tabop = true;
+                } else if (BITS == 4 && (ty == OP_TT || ty == OP_TS)) {  // 16-row base-set tables (S24)
+                    tip81<T, true>(va, r, (T)ed.x, (T)ed.y, pi);          // e [X in set] + em pi(set)
+                    st4<T>(tab + r * 4, va);
+                    if (ty == OP_TT) {
+                        tip81<T, true>(vb, r, (T)ed.z, (T)ed.w, pi);
+                        st4<T>(tab + (16 + r) * 4, vb);
+                    }
                 } else if (ty == OP_TT && r < 8) {  // two tip tables: a at [0, 16), b at [16, 32)
                     if (r < 4) tipvec<T>(va, r, (T)ed.x, (T)ed.y, pi);
                     else tipvec<T>(va, r - 4, (T)ed.z, (T)ed.w, pi);
@@ -1157,7 +1188,7 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
                 lds2(up, oa + 16u);
                 const UpBr<T, GM> ub(up, s_P);
                 const int di = (int)((ox.x >> 2) & 15u) * 4 + (int)(ox.x & 3u);  // dense (sp, type) index
-                run_op<T, DR, SI, PT, DMX, GM>(di, st, ox.x, ox.y, ox.w, cc.word((ox.x >> 6) & 2047), ub, s_tab_a,
+                run_op<T, DR, SI, PT, DMX, GM, CD>(di, st, ox.x, ox.y, ox.w, cc.word((ox.x >> 6) & 2047), ub, s_tab_a,
                                                cc, pi, scale);
             }
             const int site0 = s_begin + b * BATCH + tid * SI;
@@ -1190,12 +1221,12 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
 #endif
 }
 
-template <typename T, int DR, int SI, bool PT, int DMX, bool W, bool GM>
+template <typename T, int DR, int SI, bool PT, int DMX, bool W, bool GM, int BITS>
 __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
     extern __shared__ __align__(16) unsigned char smem_raw[];
     const int tree = blockIdx.y;
     if (a.tree_need && a.tree_need[tree] > a.need_cap) return;  // deeper tree: scored by the flat pass
-    prune_tab_body<T, DR, SI, PT, DMX, W, GM>(
+    prune_tab_body<T, DR, SI, PT, DMX, W, GM, BITS>(
         a, tree, blockIdx.x, a.sched_op + (size_t)tree * a.nops,
         reinterpret_cast<const typename Traits<T>::E4*>(a.sched_e) + (size_t)tree * a.nops, smem_raw);
 }
@@ -1228,14 +1259,14 @@ static cudaError_t launch_flat(const PruneArgs& a, int ntrees, cudaStream_t st) 
 // occupancy the kernel reaches without them (registers or base shared memory
 // bound it), so fusion never costs a resident CTA.  Cached per tree size; the
 // first call is at init (mpcgs_init scores G0), outside any graph capture.
-template <typename T, int DR, int SI, bool PT, bool GM, typename K>
+template <typename T, int DR, int SI, bool PT, bool GM, int BITS, typename K>
 static int tab_trip_cap(K kern, int nops, int need_cap) {
     if (!PT || MPCGS_NO_TRIPLETS) return 0;
     static int key[8] = {-1, -1, -1, -1, -1, -1, -1, -1}, val[8];
     const int k = nops * 16 + need_cap;
     for (int i = 0; i < 8; ++i)
         if (key[i] == k) return val[i];
-    const size_t base = tab_smem_bytes<T, DR, SI, PT, GM>(nops, need_cap, 0);
+    const size_t base = tab_smem_bytes<T, DR, SI, PT, GM, BITS>(nops, need_cap, 0);
     int dev = 0, per_sm = 0, resv = 0, optin = 0, blocks = 0;
     cudaGetDevice(&dev);
     cudaDeviceGetAttribute(&per_sm, cudaDevAttrMaxSharedMemoryPerMultiprocessor, dev);
@@ -1261,11 +1292,11 @@ static int tab_trip_cap(K kern, int nops, int need_cap) {
     return cap;
 }
 
-template <typename T, int DR, int SI, bool PT, int DMX, bool W, bool GM>
+template <typename T, int DR, int SI, bool PT, int DMX, bool W, bool GM, int BITS>
 static cudaError_t launch_tab_w(PruneArgs a, int ntrees, cudaStream_t st) {
-    auto kern = k_prune_tab<T, DR, SI, PT, DMX, W, GM>;
-    a.trip_cap = tab_trip_cap<T, DR, SI, PT, GM>(kern, a.nops, a.need_cap);
-    const size_t smem = tab_smem_bytes<T, DR, SI, PT, GM>(a.nops, a.need_cap, a.trip_cap);
+    auto kern = k_prune_tab<T, DR, SI, PT, DMX, W, GM, BITS>;
+    a.trip_cap = tab_trip_cap<T, DR, SI, PT, GM, BITS>(kern, a.nops, a.need_cap);
+    const size_t smem = tab_smem_bytes<T, DR, SI, PT, GM, BITS>(a.nops, a.need_cap, a.trip_cap);
     static size_t attr_bytes = 48 * 1024;
     if (smem > attr_bytes) {
         cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
@@ -1277,10 +1308,10 @@ static cudaError_t launch_tab_w(PruneArgs a, int ntrees, cudaStream_t st) {
     return cudaGetLastError();
 }
 
-template <typename T, int DR, int SI, bool PT, int DMX, bool GM>
+template <typename T, int DR, int SI, bool PT, int DMX, bool GM, int BITS>
 static cudaError_t launch_tab(const PruneArgs& a, int ntrees, cudaStream_t st) {
-    return a.site_w ? launch_tab_w<T, DR, SI, PT, DMX, true, GM>(a, ntrees, st)
-                    : launch_tab_w<T, DR, SI, PT, DMX, false, GM>(a, ntrees, st);
+    return a.site_w ? launch_tab_w<T, DR, SI, PT, DMX, true, GM, BITS>(a, ntrees, st)
+                    : launch_tab_w<T, DR, SI, PT, DMX, false, GM, BITS>(a, ntrees, st);
 }
 
 constexpr int PRUNE_SI_LARGE = 2;  // sites per thread for n > 128
@@ -1300,13 +1331,13 @@ inline bool product_tables(int n) {
            (size_t)MPCGS_PT_SMEM_MAX;
 }
 
-template <typename T, int SI, bool PT, bool GM>
+template <typename T, int SI, bool PT, bool GM, int BITS = 2>
 static cudaError_t launch_tab_dmx(const PruneArgs& a, int ntrees, cudaStream_t st) {
     switch (a.need_cap) {
-        case 1: case 2: case 3: case 4: return launch_tab<T, PRUNE_DR, SI, PT, 4, GM>(a, ntrees, st);
-        case 5: case 6: return launch_tab<T, PRUNE_DR, SI, PT, 6, GM>(a, ntrees, st);
-        case 7: case 8: return launch_tab<T, PRUNE_DR, SI, PT, 8, GM>(a, ntrees, st);
-        default: return launch_tab<T, PRUNE_DR, SI, PT, 10, GM>(a, ntrees, st);
+        case 1: case 2: case 3: case 4: return launch_tab<T, PRUNE_DR, SI, PT, 4, GM, BITS>(a, ntrees, st);
+        case 5: case 6: return launch_tab<T, PRUNE_DR, SI, PT, 6, GM, BITS>(a, ntrees, st);
+        case 7: case 8: return launch_tab<T, PRUNE_DR, SI, PT, 8, GM, BITS>(a, ntrees, st);
+        default: return launch_tab<T, PRUNE_DR, SI, PT, 10, GM, BITS>(a, ntrees, st);
     }
 }
 
@@ -1336,7 +1367,7 @@ cudaError_t launch_prune_typed(PruneArgs a, int ntrees, int depth, cudaStream_t 
         ++nl;
         return cudaGetLastError();
     };
-    if (a.codes2 == nullptr || !prune_uses_tables(n, sizeof(T) == 4 ? 32 : 64, GM)) {
+    if (a.codes2 == nullptr || !prune_uses_tables(n, sizeof(T) == 4 ? 32 : 64, GM, a.amb != 0)) {
         a.tree_need = nullptr;  // flat kernel for every tree
         cudaError_t e = pmats();
         if (e != cudaSuccess) return e;
@@ -1346,8 +1377,10 @@ cudaError_t launch_prune_typed(PruneArgs a, int ntrees, int depth, cudaStream_t 
     a.need_cap = prune_need_cap(n);
     const bool deep = prune_max_need(n) > a.need_cap && a.tree_need != nullptr;
     if (!deep) a.tree_need = nullptr;
-    const bool pt = product_tables<T, GM>(n);
-    cudaError_t e = (pt && !wide_sites(n)) ? launch_tab_dmx<T, PRUNE_SI_LARGE, true, GM>(a, ntrees, st)
+    const bool pt = !a.amb && product_tables<T, GM>(n);
+    cudaError_t e = a.amb ? (wide_sites(n) ? launch_tab_dmx<T, SI, false, GM, 4>(a, ntrees, st)
+                                           : launch_tab_dmx<T, PRUNE_SI_LARGE, false, GM, 4>(a, ntrees, st))
+                    : (pt && !wide_sites(n)) ? launch_tab_dmx<T, PRUNE_SI_LARGE, true, GM>(a, ntrees, st)
                     : pt ? launch_tab_dmx<T, SI, true, GM>(a, ntrees, st)
                                       : launch_tab_dmx<T, PRUNE_SI_LARGE, false, GM>(a, ntrees, st);
     nl += 1;

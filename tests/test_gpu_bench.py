@@ -36,3 +36,16 @@ def test_bench_reference_arm_cpu():
     d = _run("--impl", "reference", "--workload", "c1", "--steps", "2", "--warmup", "1", timeout=300)
     assert d["impl"] == "reference" and d["value"] > 0
     assert d["e2e"]["h2d_bytes_per_step"] == 0 and d["cpu_baseline"]["kind"] == "oracle"
+
+
+@pytest.mark.gpu
+@pytest.mark.parametrize("extra", [["--ambiguity", "0.05"], ["--model", "F84", "--kappa", "2.0"],
+                                   ["--precision", "32", "--incremental"]])
+def test_bench_variant_lines(extra):
+    """The optional workload switches each produce a valid line."""
+    d = _run("--workload", "c2", "--steps", "3", "--warmup", "3", "--cpu-seconds", "1", *extra)
+    assert d["value"] > 0 and d["gpu_launches"] > 0
+    if "--incremental" in extra:  # no flop-count fraction for incremental rescoring (bench.py)
+        assert d["roofline"]["kernel"] == "k_score_incr" and d["roofline"]["frac"] is None
+    else:
+        assert d["roofline"]["frac"] > 0
