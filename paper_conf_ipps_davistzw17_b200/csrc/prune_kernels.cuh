@@ -792,7 +792,11 @@ __host__ __device__ size_t tab_smem_bytes(int nops, int need, int trip_cap) {
 #ifdef MPCGS_MINB  // tuning builds only: min CTAs per SM (caps registers)
 #define MPCGS_TAB_BOUNDS __launch_bounds__(PRUNE_THREADS, MPCGS_MINB)
 #else
-#define MPCGS_TAB_BOUNDS __launch_bounds__(PRUNE_THREADS)
+// FP64: hold the register budget at 3 CTAs per SM (<= 168 registers).  The general
+// model (F84 / HKY85) would take 204 and fall to 2 CTAs (c5 F84 9.63 -> 8.27 ms per
+// step); the F81 kernel uses the room for scheduling (159 -> 165, 6.29 -> 6.20 ms).
+// FP32 is left free (minBlocks 0: a cap of 3 raised it from 96 to 118 registers, -0.6 %).
+#define MPCGS_TAB_BOUNDS __launch_bounds__(PRUNE_THREADS, sizeof(T) == 8 ? 3 : 0)
 #endif
 #ifdef MPCGS_PRUNE_TS  // diagnosis: setup phase cycles of CTA (0, 0), printed once per launch
 static __device__ long long g_pts[8];
