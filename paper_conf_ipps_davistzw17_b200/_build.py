@@ -63,7 +63,9 @@ def build(force: bool = False, verbose: bool = False, out: str = LIB, defines=()
         sys.stderr.write(log)
         shutil.rmtree(objdir, ignore_errors=True)
         raise RuntimeError("nvcc failed building libmpcgs.so")
-    res = subprocess.run([nvcc, "-shared", "-Xcompiler", "-fPIC", "-o", tmp, *objs, "-ldl"], capture_output=True,
+    # the link carries the arch too: without it nvcc adds an (empty) sm_52 device-link image
+    res = subprocess.run([nvcc, "-shared", "-gencode", "arch=compute_100a,code=sm_100a", "-Xcompiler", "-fPIC",
+                          "-o", tmp, *objs, "-ldl"], capture_output=True,
                          text=True)
     shutil.rmtree(objdir, ignore_errors=True)
     if res.returncode != 0:

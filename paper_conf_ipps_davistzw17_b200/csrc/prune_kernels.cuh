@@ -501,7 +501,31 @@ constexpr int OP_FUSED_SHIFT = 29;
 // followed by the TS op that joins it to tip c -- one 64x4 table of the result
 // over (x_a, x_b, x_c), built per CTA.  Type 3 is unused by the schedule encoding.
 constexpr uint32_t OP_TTT = 3u;
-constexpr int TRIP_EXTRA = 256 - 64 - 16;  // table values a fused triplet adds (64x4 vs 16x4 + 4x4)
+constexpr int TRIP_EXTRA = 256 - 64 - 16;
+// Code rows in consumption order (table kernel): the staged tip codes of a batch are
+// laid out in the order the ops read the tips (each tip is read by exactly one op, in
+// schedule order), so op i's words sit at rows k_i, k_i + 1, k_i + 2 with k_i a running
+// count -- the code-word loads no longer wait for the op record.  `tc` carries k_i.
+// Measured (interleaved A/B, profiles/r02_slot_rows_ab.txt): +3.7 % for the FP64 general
+// model on 2-bit codes at need cap 4 (n <= 64; c5 F84 8.26 -> 7.95 ms); a loss for F81
+// (FP64 -2.7 %, FP32 -5.6 %), FP32 F84 (-4.5 %), n = 128 / 256 HKY85 (-1.6 / -4 %) and
+// 4-bit codes (-2.4 %) -- so that case only.
+#ifndef MPCGS_SLOT_CODES
+#define MPCGS_SLOT_CODES 2  // 0 never, 1 always, 2 the measured case
+#endif
+template <typename T, bool GM, int DMX, typename CD>
+__host__ __device__ constexpr bool slot_rows() {
+    return MPCGS_SLOT_CODES == 1 ||
+           (MPCGS_SLOT_CODES == 2 && GM && sizeof(T) == 8 && DMX == 4 && CD::SPW == 16);
+}
+#define MPCGS_ROW_B(code, tc) (slot_rows<T, GM, DMX, CD>() ? (int)(tc) + 1 : (int)(((code) >> 17) & 2047u))
+#define MPCGS_ROW_C(tc) (slot_rows<T, GM, DMX, CD>() ? (int)(tc) + 2 : (int)(tc))
+// tips an op reads (slot advance): TT 2, TS 1 / 2 / 3 (tip / fused cherry / fused triplet),
+// SS 0, TTT 3; index = type | kind << 2 (two bits per entry)
+__device__ __forceinline__ uint32_t op_tips(uint32_t x) {
+    const uint32_t idx = (x & 3u) | (((x >> 29) & 3u) << 2);
+    return (0x00CECAC6u >> (2u * idx)) & 3u;
+}  // table values a fused triplet adds (64x4 vs 16x4 + 4x4)
 constexpr int BOUND_NEG_INF = -100000;   // ilogb of 0 (or of a subnormal): no bound
 // FP64 only: FP32's range leaves no room between checks (every op would be flagged)
 template <typename T>
@@ -623,12 +647,12 @@ struct UpBr {
 };
 
 template <typename T, int DR, int SI, bool PT, int S, int DMX, bool GM, typename CD>
-__device__ __forceinline__ void tab_tt(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, uint32_t wa,
+__device__ __forceinline__ void tab_tt(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, uint32_t tc, uint32_t wa,
                                        const UpBr<T, GM>& ub, uint32_t s_tab, const CD& c,
                                        const T (&pi)[4], int (&scale)[SI]) {
     if constexpr (S < DMX) {
         constexpr int EB = 4 * sizeof(T);
-        const uint32_t wb = c.word((code >> 17) & 2047);
+        const uint32_t wb = c.word(MPCGS_ROW_B(code, tc));
         const uint32_t base = s_tab + (toff & ~TAB_CHECK);
         T v[SI][4];
         if constexpr (PT) {  // 16x4 table of the cherry, entry 4 x_a + x_b: branch_up(tip_a (.) tip_b)
@@ -669,8 +693,8 @@ __device__ __forceinline__ void tab_ttt(Stack<T, DR, SI>& st, uint32_t code, uin
                                         const T (&pi)[4], int (&scale)[SI]) {
     if constexpr (PT && S < DMX) {
         constexpr int EB = 4 * sizeof(T);
-        const uint32_t wb = c.word((code >> 17) & 2047);
-        const uint32_t wc = c.word((int)tc);
+        const uint32_t wb = c.word(MPCGS_ROW_B(code, tc));
+        const uint32_t wc = c.word(MPCGS_ROW_C(tc));
         const uint32_t base = s_tab + (toff & ~TAB_CHECK);
         T v[SI][4];
         const uint32_t ix = (c.lanes(wa) << 4) + (c.lanes(wb) << 2) + c.lanes(wc);  // entry 16 x_a + 4 x_b + x_c
@@ -703,8 +727,8 @@ __device__ __forceinline__ void tab_ts(Stack<T, DR, SI>& st, uint32_t code, uint
         uint32_t la = c.lanes(wa);
         const uint32_t kind = (code >> OP_FUSED_SHIFT) & 3u;
         if (kind != 0u) {
-            la = (la << 2) + c.lanes(c.word((code >> 17) & 2047));
-            if (kind == 2u) la = (la << 2) + c.lanes(c.word((int)tc));
+            la = (la << 2) + c.lanes(c.word(MPCGS_ROW_B(code, tc)));
+            if (kind == 2u) la = (la << 2) + c.lanes(c.word(MPCGS_ROW_C(tc)));
         }
         T v[SI][4];
 #pragma unroll
@@ -749,7 +773,7 @@ __device__ __forceinline__ void tab_ss(Stack<T, DR, SI>& st, uint32_t code, cons
 }
 
 #define MPCGS_TABCASE(S)                                                                          \
-    case 4 * (S) + 0: tab_tt<T, DR, SI, PT, S, DMX, GM, CD>(st, code, toff, wa, ub, s_tab, cc, pi, scale); break;       \
+    case 4 * (S) + 0: tab_tt<T, DR, SI, PT, S, DMX, GM, CD>(st, code, toff, tc, wa, ub, s_tab, cc, pi, scale); break;       \
     case 4 * (S) + 1: tab_ts<T, DR, SI, S, DMX, GM, CD>(st, code, toff, tc, wa, ub, s_tab, cc, pi, scale); break; \
     case 4 * (S) + 2: tab_ss<T, DR, SI, S, DMX, GM>(st, code, ub, pi, scale); break;                      \
     case 4 * (S) + 3: tab_ttt<T, DR, SI, PT, S, DMX, GM, CD>(st, code, toff, tc, wa, ub, s_tab, cc, pi, scale); break;
@@ -786,7 +810,8 @@ __host__ __device__ size_t tab_smem_bytes(int nops, int need, int trip_cap) {
            align16(sizeof(T) * ((PT ? 32 : (BITS == 4 ? 64 : 16)) * (size_t)n + (size_t)TRIP_EXTRA * (PT ? trip_cap : 0))) +
            align16(sizeof(OpRec<T>) * nops) + 2 * align16(Codes<SI, BITS>::buf_bytes(n)) +
            sizeof(T) * (size_t)spill * SI * 4 * PRUNE_THREADS +
-           align16(sizeof(int) * 2 * (size_t)nops) + align16(sizeof(int) * (size_t)nops) + 64 * sizeof(int);
+           align16(sizeof(int) * 2 * (size_t)nops) + align16(sizeof(int) * (size_t)nops) +
+           align16(sizeof(int) * (size_t)(nops + 1)) + 64 * sizeof(int);
 }
 
 #ifdef MPCGS_MINB  // tuning builds only: min CTAs per SM (caps registers)
@@ -833,6 +858,7 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
     int* s_d = reinterpret_cast<int*>(reinterpret_cast<unsigned char*>(s_spill) +
                                       sizeof(T) * (size_t)spill_lv * SI * 4 * PRUNE_THREADS);
     int* s_tl = s_d + align16(sizeof(int) * 2 * (size_t)nops) / sizeof(int);  // original codes, then check flags
+    int* s_pos = s_tl + align16(sizeof(int) * (size_t)nops) / sizeof(int);     // tip -> code row (MPCGS_SLOT_CODES)
     __shared__ int s_nc;  // compacted op count
 
     const int tid = threadIdx.x;
@@ -848,11 +874,12 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
         const uint32_t* src = a.codes2 + site0 / CD::SPW;
         for (int c = tid; c < n * CH; c += PRUNE_THREADS) {
             const int tip = c / CH, q = c - tip * CH;
-            cp_async16(dst + ((size_t)tip * WB + q * 4) * 4, src + (size_t)tip * a.W2 + q * 4);
+            const int row = slot_rows<T, GM, DMX, CD>() ? s_pos[tip] : tip;
+            cp_async16(dst + ((size_t)row * WB + q * 4) * 4, src + (size_t)tip * a.W2 + q * 4);
         }
         cp_async_commit();
     };
-    if (nb > 0) issue(0, 0);
+    if (!slot_rows<T, GM, DMX, CD>() && nb > 0) issue(0, 0);  // (slot rows: after the scan below lays them out)
 
     // 1. schedule, branch data and the per-child bounds d (mark_checks, fusion guard)
     const T pi[4] = {(T)a.pi[0], (T)a.pi[1], (T)a.pi[2], (T)a.pi[3]};
@@ -889,7 +916,7 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
     // 2. warp 0: fuse the first trip_cap (TT, TS) pairs, compact the op list and
     //    lay out the tables (exclusive scans over the original ops)
     if (tid < 32) {
-        uint32_t c_keep = 0, c_size = 0, c_cand = 0, prev_start = 0;
+        uint32_t c_keep = 0, c_size = 0, c_cand = 0, prev_start = 0, c_rows = 0;
         for (int base = 0; base < nops; base += 32) {
             const int i = base + tid;
             uint32_t code = 0, ty = 2, tyn = 2;
@@ -918,6 +945,19 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
                 if (tid >= o) x += y;
             }
             const uint32_t tc = (i + 1 < nops) ? ((s_code[i + 1] >> 6) & 2047u) : 0u;
+            if (slot_rows<T, GM, DMX, CD>()) {  // code rows in consumption order: TT reads (a, b), TS reads a
+                const uint32_t nt = i < nops ? (ty == OP_TT ? 2u : (ty == OP_TS ? 1u : 0u)) : 0u;
+                uint32_t y = nt;
+#pragma unroll
+                for (int o = 1; o < 32; o <<= 1) {
+                    const uint32_t z = __shfl_up_sync(0xffffffffu, y, o);
+                    if (tid >= o) y += z;
+                }
+                const uint32_t row = c_rows + y - nt;
+                if (nt >= 1u) s_pos[(code >> 6) & 2047u] = (int)row;
+                if (nt == 2u) s_pos[(code >> 17) & 2047u] = (int)row + 1;
+                c_rows += __shfl_sync(0xffffffffu, y, 31);
+            }
             __syncwarp();
             if (keep) {
                 const uint32_t cx = start ? ((code & ~3u) | OP_TTT) : code;
@@ -932,6 +972,7 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
     }
     __syncthreads();
     PTS(3);
+    if (slot_rows<T, GM, DMX, CD>() && nb > 0) issue(0, 0);
     const int nops_c = s_nc;
     // 3. sparse checks (FP64): warp 1 walks the bounds while the others build the tables
     unsigned char* s_chk = reinterpret_cast<unsigned char*>(s_tl);  // s_code is dead after the scan
@@ -1185,15 +1226,19 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
             int scale[SI];
 #pragma unroll
             for (int k = 0; k < SI; ++k) scale[k] = 0;
+            uint32_t krow = 0;  // code row of the op's first tip (MPCGS_SLOT_CODES)
             for (int op = 0; op < nops_run; ++op) {
                 const uint32_t oa = s_opc_a + (uint32_t)op * (uint32_t)sizeof(OpRec<T>);
+                const uint32_t wa = slot_rows<T, GM, DMX, CD>() ? cc.word((int)krow) : 0u;  // issued beside the record load
                 const uint4 ox = lds_u4(oa);
                 T up[2];
                 lds2(up, oa + 16u);
                 const UpBr<T, GM> ub(up, s_P);
                 const int di = (int)((ox.x >> 2) & 15u) * 4 + (int)(ox.x & 3u);  // dense (sp, type) index
-                run_op<T, DR, SI, PT, DMX, GM, CD>(di, st, ox.x, ox.y, ox.w, cc.word((ox.x >> 6) & 2047), ub, s_tab_a,
-                                               cc, pi, scale);
+                run_op<T, DR, SI, PT, DMX, GM, CD>(di, st, ox.x, ox.y, slot_rows<T, GM, DMX, CD>() ? krow : ox.w,
+                                                   slot_rows<T, GM, DMX, CD>() ? wa : cc.word((ox.x >> 6) & 2047), ub, s_tab_a,
+                                                   cc, pi, scale);
+                krow += op_tips(ox.x);
             }
             const int site0 = s_begin + b * BATCH + tid * SI;
 #pragma unroll
