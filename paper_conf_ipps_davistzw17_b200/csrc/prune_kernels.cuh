@@ -511,12 +511,11 @@ constexpr int TRIP_EXTRA = 256 - 64 - 16;
 // (FP64 -2.7 %, FP32 -5.6 %), FP32 F84 (-4.5 %), n = 128 / 256 HKY85 (-1.6 / -4 %) and
 // 4-bit codes (-2.4 %) -- so that case only.
 #ifndef MPCGS_SLOT_CODES
-#define MPCGS_SLOT_CODES 2  // 0 never, 1 always, 2 the measured case
+#define MPCGS_SLOT_CODES 1  // 0: off (tuning builds)
 #endif
 template <typename T, bool GM, int DMX, typename CD>
 __host__ __device__ constexpr bool slot_rows() {
-    return MPCGS_SLOT_CODES == 1 ||
-           (MPCGS_SLOT_CODES == 2 && GM && sizeof(T) == 8 && DMX == 4 && CD::SPW == 16);
+    return MPCGS_SLOT_CODES && GM && sizeof(T) == 8 && DMX == 4 && CD::SPW == 16;
 }
 #define MPCGS_ROW_B(code, tc) (slot_rows<T, GM, DMX, CD>() ? (int)(tc) + 1 : (int)(((code) >> 17) & 2047u))
 #define MPCGS_ROW_C(tc) (slot_rows<T, GM, DMX, CD>() ? (int)(tc) + 2 : (int)(tc))
@@ -811,7 +810,8 @@ __host__ __device__ size_t tab_smem_bytes(int nops, int need, int trip_cap) {
            align16(sizeof(OpRec<T>) * nops) + 2 * align16(Codes<SI, BITS>::buf_bytes(n)) +
            sizeof(T) * (size_t)spill * SI * 4 * PRUNE_THREADS +
            align16(sizeof(int) * 2 * (size_t)nops) + align16(sizeof(int) * (size_t)nops) +
-           align16(sizeof(int) * (size_t)(nops + 1)) + 64 * sizeof(int);
+           (GM && sizeof(T) == 8 && BITS == 2 ? align16(sizeof(int) * (size_t)(nops + 1)) : 0) +  // slot rows
+           64 * sizeof(int);
 }
 
 #ifdef MPCGS_MINB  // tuning builds only: min CTAs per SM (caps registers)
@@ -858,7 +858,9 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
     int* s_d = reinterpret_cast<int*>(reinterpret_cast<unsigned char*>(s_spill) +
                                       sizeof(T) * (size_t)spill_lv * SI * 4 * PRUNE_THREADS);
     int* s_tl = s_d + align16(sizeof(int) * 2 * (size_t)nops) / sizeof(int);  // original codes, then check flags
-    int* s_pos = s_tl + align16(sizeof(int) * (size_t)nops) / sizeof(int);     // tip -> code row (MPCGS_SLOT_CODES)
+    // tip -> code row (slot_rows only: reserved for FP64 general-model 2-bit kernels; every
+    // byte here costs the others triplet tables, FP32 c5 -3.8 % with it)
+    int* s_pos = s_tl + align16(sizeof(int) * (size_t)nops) / sizeof(int);
     __shared__ int s_nc;  // compacted op count
 
     const int tid = threadIdx.x;
