@@ -60,6 +60,22 @@ __device__ __forceinline__ void branch(T (&r)[4], T e, T em, const T (&pi)[4]) {
     r[3] = fma(e, r[3], t);
 }
 
+// The same branch divided by e (a per-branch constant, the same at every site):
+// branch(L)_X / e = L_X + r (pi . L), r = em / e = e^{ut} - 1.  One FP instruction
+// per site fewer than branch(); the table kernel adds sum ln e per site back once
+// per genealogy (prune_kernels.cuh, unit_branch).
+template <typename T>
+__device__ __forceinline__ void branch_unit(T (&v)[4], T r, const T (&pi)[4]) {
+    T s = pi[0] * v[0];
+    s = fma(pi[1], v[1], s);
+    s = fma(pi[2], v[2], s);
+    s = fma(pi[3], v[3], s);
+    v[0] = fma(r, s, v[0]);
+    v[1] = fma(r, s, v[1]);
+    v[2] = fma(r, s, v[2]);
+    v[3] = fma(r, s, v[3]);
+}
+
 // tip(x)_X = P_{X,x}(t) = e [X==x] + em pi_x   (tips are indicators, L673-676)
 template <typename T>
 __device__ __forceinline__ void tipvec(T (&r)[4], int x, T e, T em, const T (&pi)[4]) {
@@ -246,13 +262,13 @@ struct ExactScratch {
 // Per-genealogy accumulator in device memory: [0] lo, [1] hi, [2] flags (zero on entry;
 // reset by the CTA that completes the genealogy).
 // Block-reduce v (exactly), add it to acc with 64-bit atomics (carry from the low
-// word's old value), and let the last of `tiles` CTAs write the double to *out.
+// word's old value), and let the last of `tiles` CTAs write the double (+ add) to *out.
 // scratch: shared memory of >= 3 * NT / 32 + 1 words, free for the call (the table
 // kernel passes its tip-code staging buffers, so the commit adds no static shared
 // memory that would cost it a fused triplet table).
 template <int NT>
 __device__ __forceinline__ void exact_commit(Exact128 v, unsigned long long* acc, unsigned* cnt, int tiles,
-                                             double* out, unsigned long long* scratch) {
+                                             double* out, unsigned long long* scratch, double add = 0.0) {
     unsigned long long* s_lo = scratch;
     long long* s_hi = reinterpret_cast<long long*>(scratch + NT / 32);
     unsigned long long* s_fl = scratch + 2 * (NT / 32);
@@ -288,7 +304,7 @@ __device__ __forceinline__ void exact_commit(Exact128 v, unsigned long long* acc
         __threadfence();
         const volatile unsigned long long* va = acc;
         const unsigned long long lo = va[0], hi = va[1], fl = va[2];
-        *out = exact_to_double(lo, (long long)hi, (unsigned)fl);
+        *out = exact_to_double(lo, (long long)hi, (unsigned)fl) + add;  // add: the same in every CTA of the tree
         acc[0] = 0ull;
         acc[1] = 0ull;
         acc[2] = 0ull;

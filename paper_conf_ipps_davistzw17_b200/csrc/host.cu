@@ -709,6 +709,7 @@ PruneArgs prune_args(mpcgs_ctx* c, int ntrees, double* out, int out_first, int o
     a.codes = c->s.codes;
     a.codes2 = c->codes2;
     a.site_w = c->s.site_w;
+    a.sum_w = (double)c->L_orig;  // pattern counts sum to the alignment's columns
     a.W2 = codes2_words(c->L) * (c->s.amb ? 2 : 1);  // 4-bit codes with ambiguity data
     a.Lpad = c->Lpad;
     a.L = c->L;

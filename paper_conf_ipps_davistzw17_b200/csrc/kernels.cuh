@@ -35,6 +35,7 @@ struct PruneArgs {
     // unit_sites sites each (balanced; tile_range below); sites_per_cta = the largest tile
     int tiles, sites_per_cta, units, unit_sites;
     const double* site_w;      // [L] pattern counts (compressed sites, f3) or nullptr
+    double sum_w;              // sum of the site weights (= alignment columns)
     const int32_t* tree_need;  // [ntrees] register need of each tree's schedule (nullable)
     int need_cap;              // set by launch_prune: largest need the table kernel serves
     int trip_cap;              // set by launch_prune: fused triplets per tree (table kernel)

@@ -365,6 +365,36 @@ __device__ __forceinline__ void lds4(float (&r)[4], uint32_t a) {
     asm volatile("ld.shared.v4.f32 {%0, %1, %2, %3}, [%4];\n" : "=f"(r[0]), "=f"(r[1]), "=f"(r[2]), "=f"(r[3]) : "r"(a));
 }
 
+// FP64 tables in split-half layout: a table of E entries stores the first halves
+// {v0, v1} of its entries (16 B each), then the second halves {v2, v3}.  A warp's
+// 16-byte loads of data-dependent entries then spread over all 8 bank groups of a
+// 128-byte row (contiguous 32-byte entries put every first half in an even group:
+// about 1.4x the shared-memory wavefronts on random 16- and 64-entry gathers).
+#ifndef MPCGS_SPLITTAB
+#define MPCGS_SPLITTAB 1
+#endif
+template <typename T>
+__host__ __device__ constexpr bool split_tab() { return MPCGS_SPLITTAB && sizeof(T) == 8; }
+template <typename T>
+__device__ __forceinline__ void tab_st(T* tab, int E, int i, const T (&v)[4]) {
+    if constexpr (split_tab<T>()) {
+        reinterpret_cast<double2*>(tab)[i] = make_double2(v[0], v[1]);
+        reinterpret_cast<double2*>(tab)[E + i] = make_double2(v[2], v[3]);
+    } else {
+        st4<T>(tab + 4 * i, v);
+    }
+}
+// entry of a table at byte address base: eo = the entry's index x 16 (split) or x 4 sizeof(T)
+__device__ __forceinline__ void tab_ld(double (&r)[4], uint32_t a, uint32_t E) {
+    if constexpr (split_tab<double>()) {
+        asm volatile("ld.shared.v2.f64 {%0, %1}, [%2];\n" : "=d"(r[0]), "=d"(r[1]) : "r"(a));
+        asm volatile("ld.shared.v2.f64 {%0, %1}, [%2];\n" : "=d"(r[2]), "=d"(r[3]) : "r"(a + 16u * E));
+    } else {
+        lds4(r, a);
+    }
+}
+__device__ __forceinline__ void tab_ld(float (&r)[4], uint32_t a, uint32_t) { lds4(r, a); }
+
 template <typename T, int SI>
 __device__ __forceinline__ void rescale_sites(T (&v)[SI][4], int (&scale)[SI]) {
     bool any = false;
@@ -530,6 +560,15 @@ constexpr int BOUND_NEG_INF = -100000;   // ilogb of 0 (or of a subnormal): no b
 template <typename T>
 __host__ __device__ constexpr bool sparse_checks() { return MPCGS_SPARSE && sizeof(T) == 8; }
 
+// unit-diagonal F81 branches in the table kernel (FP64; see prune_tab_body)
+#ifndef MPCGS_UNITBR
+#define MPCGS_UNITBR 1
+#endif
+template <typename T, bool GM>
+__host__ __device__ constexpr bool unit_branch() {
+    return MPCGS_UNITBR && !GM && sizeof(T) == 8;
+}
+
 template <typename T>
 struct Bounds;
 template <>
@@ -627,7 +666,9 @@ __device__ void mark_checks(const OpRec<T>* s_opc, const int* s_d, unsigned char
 // enough to need a rescale (TAB_CHECK, rare): then the raw entry is loaded,
 // checked and transformed per site.  The up branch of the root op is the
 // identity (e = 1, em = 0 / P = I), which leaves the root vector unchanged.
-template <typename T, bool GM>
+// U (unit-diagonal F81 branches, see unit_branch below): the record holds {1, r} with
+// r = em / e, and the branch is v + r (pi . v) -- the e multiply is dropped.
+template <typename T, bool GM, bool U = false>
 struct UpBr {
     std::conditional_t<GM, const T*, T> e;
     T em;
@@ -641,23 +682,24 @@ struct UpBr {
     }
     __device__ __forceinline__ void apply(T (&v)[4], const T (&pi)[4]) const {
         if constexpr (GM) gm_branch_c<T>(v, e, pi);  // e -> the structured branch record
+        else if constexpr (U) branch_unit<T>(v, em, pi);
         else branch<T>(v, e, em, pi);
     }
 };
 
-template <typename T, int DR, int SI, bool PT, int S, int DMX, bool GM, typename CD>
+template <typename T, int DR, int SI, bool PT, int S, int DMX, bool GM, typename CD, typename UB>
 __device__ __forceinline__ void tab_tt(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, uint32_t tc, uint32_t wa,
-                                       const UpBr<T, GM>& ub, uint32_t s_tab, const CD& c,
+                                       const UB& ub, uint32_t s_tab, const CD& c,
                                        const T (&pi)[4], int (&scale)[SI]) {
     if constexpr (S < DMX) {
-        constexpr int EB = 4 * sizeof(T);
+        constexpr int EB = split_tab<T>() ? 16 : 4 * sizeof(T);  // entry stride (split-half tables: 16)
         const uint32_t wb = c.word(MPCGS_ROW_B(code, tc));
         const uint32_t base = s_tab + (toff & ~TAB_CHECK);
         T v[SI][4];
         if constexpr (PT) {  // 16x4 table of the cherry, entry 4 x_a + x_b: branch_up(tip_a (.) tip_b)
             const uint32_t ix = (c.lanes(wa) << 2) + c.lanes(wb);
 #pragma unroll
-            for (int k = 0; k < SI; ++k) lds4(v[k], base + c.template off<EB>(ix, k));
+            for (int k = 0; k < SI; ++k) tab_ld(v[k], base + c.template off<EB>(ix, k), 16u);
             if (toff & TAB_CHECK) {  // raw table: check, then the up branch per site
                 rescale_sites<T, SI>(v, scale);
 #pragma unroll
@@ -668,8 +710,8 @@ __device__ __forceinline__ void tab_tt(Stack<T, DR, SI>& st, uint32_t code, uint
 #pragma unroll
             for (int k = 0; k < SI; ++k) {
                 T w[4];
-                lds4(v[k], base + c.template off<EB>(la, k));
-                lds4(w, base + 4u * (CD::LM + 1u) * (uint32_t)sizeof(T) + c.template off<EB>(lb, k));  // table b after a
+                tab_ld(v[k], base + c.template off<EB>(la, k), CD::LM + 1u);
+                tab_ld(w, base + 4u * (CD::LM + 1u) * (uint32_t)sizeof(T) + c.template off<EB>(lb, k), CD::LM + 1u);  // table b after a
 #pragma unroll
                 for (int i = 0; i < 4; ++i) v[k][i] *= w[i];
             }
@@ -686,19 +728,19 @@ __device__ __forceinline__ void tab_tt(Stack<T, DR, SI>& st, uint32_t code, uint
 }
 
 // fused triplet: one lookup in the 64x4 table of branch_up(tip(c) (.) branch(tip(a) (.) tip(b)))
-template <typename T, int DR, int SI, bool PT, int S, int DMX, bool GM, typename CD>
+template <typename T, int DR, int SI, bool PT, int S, int DMX, bool GM, typename CD, typename UB>
 __device__ __forceinline__ void tab_ttt(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, uint32_t tc,
-                                        uint32_t wa, const UpBr<T, GM>& ub, uint32_t s_tab, const CD& c,
+                                        uint32_t wa, const UB& ub, uint32_t s_tab, const CD& c,
                                         const T (&pi)[4], int (&scale)[SI]) {
     if constexpr (PT && S < DMX) {
-        constexpr int EB = 4 * sizeof(T);
+        constexpr int EB = split_tab<T>() ? 16 : 4 * sizeof(T);
         const uint32_t wb = c.word(MPCGS_ROW_B(code, tc));
         const uint32_t wc = c.word(MPCGS_ROW_C(tc));
         const uint32_t base = s_tab + (toff & ~TAB_CHECK);
         T v[SI][4];
         const uint32_t ix = (c.lanes(wa) << 4) + (c.lanes(wb) << 2) + c.lanes(wc);  // entry 16 x_a + 4 x_b + x_c
 #pragma unroll
-        for (int k = 0; k < SI; ++k) lds4(v[k], base + c.template off<EB>(ix, k));
+        for (int k = 0; k < SI; ++k) tab_ld(v[k], base + c.template off<EB>(ix, k), 64u);
         if (toff & TAB_CHECK) {
             rescale_sites<T, SI>(v, scale);
 #pragma unroll
@@ -716,15 +758,16 @@ __device__ __forceinline__ void tab_ttt(Stack<T, DR, SI>& st, uint32_t code, uin
 // Fused (OP_FUSED kind 1 / 2): a cherry / triplet table op and the SS that merges
 // its result into the stack top, v = top (.) table(x_a, x_b[, x_c]) -- the table
 // already carries the cherry's branch into the SS, the op record the SS's up branch.
-template <typename T, int DR, int SI, int S, int DMX, bool GM, typename CD>
+template <typename T, int DR, int SI, int S, int DMX, bool GM, typename CD, typename UB>
 __device__ __forceinline__ void tab_ts(Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, uint32_t tc,
-                                       uint32_t wa, const UpBr<T, GM>& ub, uint32_t s_tab, const CD& c,
+                                       uint32_t wa, const UB& ub, uint32_t s_tab, const CD& c,
                                        const T (&pi)[4], int (&scale)[SI]) {
     if constexpr (S >= 1 && S <= DMX) {
-        constexpr int EB = 4 * sizeof(T);
+        constexpr int EB = split_tab<T>() ? 16 : 4 * sizeof(T);
         const uint32_t base = s_tab + (toff & ~TAB_CHECK);
         uint32_t la = c.lanes(wa);
         const uint32_t kind = (code >> OP_FUSED_SHIFT) & 3u;
+        const uint32_t E = (CD::LM + 1u) << (2u * kind);  // tip 4 (16 base sets), cherry 16, triplet 64
         if (kind != 0u) {
             la = (la << 2) + c.lanes(c.word(MPCGS_ROW_B(code, tc)));
             if (kind == 2u) la = (la << 2) + c.lanes(c.word(MPCGS_ROW_C(tc)));
@@ -733,7 +776,7 @@ __device__ __forceinline__ void tab_ts(Stack<T, DR, SI>& st, uint32_t code, uint
 #pragma unroll
         for (int k = 0; k < SI; ++k) {
             T tip[4];
-            lds4(tip, base + c.template off<EB>(la, k));
+            tab_ld(tip, base + c.template off<EB>(la, k), E);
             st.template get<S - 1>(k, v[k]);
 #pragma unroll
             for (int i = 0; i < 4; ++i) v[k][i] *= tip[i];
@@ -748,8 +791,8 @@ __device__ __forceinline__ void tab_ts(Stack<T, DR, SI>& st, uint32_t code, uint
 }
 
 // two stack entries (each already carrying its branch): v = second (.) top
-template <typename T, int DR, int SI, int S, int DMX, bool GM>
-__device__ __forceinline__ void tab_ss(Stack<T, DR, SI>& st, uint32_t code, const UpBr<T, GM>& ub,
+template <typename T, int DR, int SI, int S, int DMX, bool GM, typename UB>
+__device__ __forceinline__ void tab_ss(Stack<T, DR, SI>& st, uint32_t code, const UB& ub,
                                        const T (&pi)[4], int (&scale)[SI]) {
     if constexpr (S >= 2 && S <= DMX) {
         T v[SI][4];
@@ -782,9 +825,9 @@ __device__ __forceinline__ void tab_ss(Stack<T, DR, SI>& st, uint32_t code, cons
 #define MPCGS_CASES_10 MPCGS_CASES_8 MPCGS_TABCASE(9) MPCGS_TABCASE(10)
 
 // one op for SI sites; the switch only has the (sp, type) labels a DMX-level tree can use
-template <typename T, int DR, int SI, bool PT, int DMX, bool GM, typename CD>
+template <typename T, int DR, int SI, bool PT, int DMX, bool GM, typename CD, typename UB>
 __device__ __forceinline__ void run_op(int di, Stack<T, DR, SI>& st, uint32_t code, uint32_t toff, uint32_t tc,
-                                       uint32_t wa, const UpBr<T, GM>& ub, uint32_t s_tab, const CD& cc,
+                                       uint32_t wa, const UB& ub, uint32_t s_tab, const CD& cc,
                                        const T (&pi)[4], int (&scale)[SI]) {
     if constexpr (DMX <= 4) {
         switch (di) { MPCGS_CASES_4 default: __builtin_unreachable(); }
@@ -887,6 +930,7 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
     const T pi[4] = {(T)a.pi[0], (T)a.pi[1], (T)a.pi[2], (T)a.pi[3]};
     const T pimin = min(min(pi[0], pi[1]), min(pi[2], pi[3]));
     uint32_t* s_code = reinterpret_cast<uint32_t*>(s_tl);  // original codes (s_tl is filled after the scan)
+    double lne = 0.0;  // unit branches: this thread's sum of ln e over its ops' two child branches
     for (int i = tid; i < nops; i += PRUNE_THREADS) {
         s_code[i] = gop[i];
         if constexpr (!GM) {  // d = em pi_min (Eq. 20)
@@ -895,6 +939,37 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
             const int lp = Bounds<T>::ilogb(pimin);
             s_d[2 * i] = Bounds<T>::ilogb((T)ed.y) + lp;
             s_d[2 * i + 1] = Bounds<T>::ilogb((T)ed.w) + lp;
+            if constexpr (unit_branch<T, GM>()) lne += log((double)ed.x) + log((double)ed.z);
+        }
+    }
+    // Unit-diagonal branches (F81, FP64): every branch b of the tree is applied divided
+    // by its e_b, so a vector carries the factor 1 / prod e_b of the branches below it
+    // and the root 1 / prod_b e_b, the same at every site: ln L_s = ln(pi . root_s) +
+    // scale_s ln 2 + C with C = sum_b ln e_b = -u (tree length), added once per tree
+    // (exact_commit).  Those factors only enlarge vectors (the S5 lower bounds stay
+    // valid); the form is used while they cannot overflow: -C / ln 2 <= 900 - n bits
+    // (a vector of the standard form is < 2^(n-1) after power-of-two rescales), else
+    // the tree keeps the standard branch.  C is reduced in a fixed order, so every CTA
+    // of a tree (any tiling, any world size) adds the same double (P22).
+    bool unit = false;
+    double lnC = 0.0;
+    if constexpr (unit_branch<T, GM>()) {
+        __shared__ double s_lne[PRUNE_THREADS / 32];
+#pragma unroll
+        for (int o = 16; o > 0; o >>= 1) lne += __shfl_down_sync(0xffffffffu, lne, o);
+        if ((tid & 31) == 0) s_lne[tid >> 5] = lne;
+        __syncthreads();
+        lnC = s_lne[0];
+#pragma unroll
+        for (int w = 1; w < PRUNE_THREADS / 32; ++w) lnC += s_lne[w];
+        unit = -lnC * 1.4426950408889634 <= (double)(900 - n);  // false for -inf / NaN
+        if (unit) {
+            for (int i = tid; i < nops; i += PRUNE_THREADS) {
+                const E4 ed = s_e[i];
+                s_e[i] = make_double4(1.0, ed.y / ed.x, 1.0, ed.w / ed.z);  // {1, r = em / e} per side
+            }
+        } else {
+            lnC = 0.0;
         }
     }
     if constexpr (GM) {  // {C_a, C_b} of every op from its branch lengths {t_a, 0, t_b, 0}; d = min_XY P_XY(t)
@@ -1057,17 +1132,17 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
                             }
                     };
                     setcol(va, Ca, r);
-                    st4<T>(tab + r * 4, va);
+                    tab_st<T>(tab, 16, r, va);
                     if (ty == OP_TT) {  // table b after table a
                         setcol(vb, Ca + GMC, r);
-                        st4<T>(tab + (16 + r) * 4, vb);
+                        tab_st<T>(tab + 16 * 4, 16, r, vb);
                     }
                 } else if (ty == OP_TT && r < 8) {
                     gm_col_c<T>(va, Ca + (r < 4 ? 0 : GMC), r & 3, pi);
-                    st4<T>(tab + r * 4, va);
+                    tab_st<T>(tab + (r & 4) * 4, 4, r & 3, va);
                 } else if (ty == OP_TS && r < 4) {
                     gm_col_c<T>(va, Ca, r, pi);
-                    st4<T>(tab + r * 4, va);
+                    tab_st<T>(tab, 4, r, va);
                 } else if (ty == OP_TTT) {  // op o: C_a, C_b; op o+1: C of tip c, C of the cherry's branch
                     const T* Cc = Ca + 2 * GMC;
                     gm_col_c<T>(va, Ca, r >> 2, pi);
@@ -1094,18 +1169,18 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
                     tabop = true;
                 } else if (BITS == 4 && (ty == OP_TT || ty == OP_TS)) {  // 16-row base-set tables (S24)
                     tip81<T, true>(va, r, (T)ed.x, (T)ed.y, pi);          // e [X in set] + em pi(set)
-                    st4<T>(tab + r * 4, va);
+                    tab_st<T>(tab, 16, r, va);
                     if (ty == OP_TT) {
                         tip81<T, true>(vb, r, (T)ed.z, (T)ed.w, pi);
-                        st4<T>(tab + (16 + r) * 4, vb);
+                        tab_st<T>(tab + 16 * 4, 16, r, vb);
                     }
                 } else if (ty == OP_TT && r < 8) {  // two tip tables: a at [0, 16), b at [16, 32)
                     if (r < 4) tipvec<T>(va, r, (T)ed.x, (T)ed.y, pi);
                     else tipvec<T>(va, r - 4, (T)ed.z, (T)ed.w, pi);
-                    st4<T>(tab + r * 4, va);
+                    tab_st<T>(tab + (r & 4) * 4, 4, r & 3, va);
                 } else if (ty == OP_TS && r < 4) {
                     tipvec<T>(va, r, (T)ed.x, (T)ed.y, pi);
-                    st4<T>(tab + r * 4, va);
+                    tab_st<T>(tab, 4, r, va);
                 } else if (ty == OP_TTT) {
                     const E4 e1 = s_e[ox.z + 1];
                     tipvec<T>(va, r >> 2, (T)ed.x, (T)ed.y, pi);
@@ -1130,7 +1205,6 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
         const unsigned m = __ballot_sync(0xffffffffu, small);
         const bool raw = ((m >> (tid & 16)) & 0xffffu) != 0u;
         if (tabop) {
-            T* row = tab + r * ne * 4;
             if (raw) {
                 if (r == 0) s_opc[op].h.y |= TAB_CHECK;
             } else {
@@ -1141,7 +1215,7 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
             }
 #pragma unroll
             for (int e = 0; e < 4; ++e)
-                if (e < ne) st4<T>(row + 4 * e, v[e]);
+                if (e < ne) tab_st<T>(tab, ne == 4 ? 64 : 16, r * ne + e, v[e]);  // cherry 16, triplet 64 entries
         }
     }
     // the check flags are merged into the op codes after this pass (which reads the
@@ -1198,8 +1272,11 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
     PTS(6);
     }
 
-    SiteAcc<W> acc;
     Exact128 ex;
+    // the batch loop, instantiated for the unit-diagonal and the standard branch form
+    auto batches = [&](auto unit_tag) {
+    constexpr bool U = decltype(unit_tag)::value;
+    SiteAcc<W> acc;
     Stack<T, DR, SI> st;
     st.sm = smem_addr(s_spill + tid);
 #pragma unroll
@@ -1235,7 +1312,7 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
                 const uint4 ox = lds_u4(oa);
                 T up[2];
                 lds2(up, oa + 16u);
-                const UpBr<T, GM> ub(up, s_P);
+                const UpBr<T, GM, U> ub(up, s_P);
                 const int di = (int)((ox.x >> 2) & 15u) * 4 + (int)(ox.x & 3u);  // dense (sp, type) index
                 run_op<T, DR, SI, PT, DMX, GM, CD>(di, st, ox.x, ox.y, slot_rows<T, GM, DMX, CD>() ? krow : ox.w,
                                                    slot_rows<T, GM, DMX, CD>() ? wa : cc.word((ox.x >> 6) & 2047), ub, s_tab_a,
@@ -1259,11 +1336,18 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
         ex.add(acc.total());
         acc.reset();
     }
+    };
+    if constexpr (unit_branch<T, GM>()) {
+        if (unit) batches(std::true_type{});
+        else batches(std::false_type{});
+    } else {
+        batches(std::false_type{});
+    }
     // the code staging buffers are free now (the last batch ended with a barrier)
     PTS(7);
     exact_commit<PRUNE_THREADS>(ex, a.tree_acc + 4 * (size_t)tree, a.tile_cnt + tree, a.tiles,
                                 a.out + (size_t)(a.out_first + tree) * a.out_stride,
-                                reinterpret_cast<unsigned long long*>(s_cod));
+                                reinterpret_cast<unsigned long long*>(s_cod), lnC * a.sum_w);
 #ifdef MPCGS_PRUNE_TS
     if (threadIdx.x == 0 && blockIdx.x == 0 && blockIdx.y == 0 && (clock64() & 7) == 0)
         printf("prune setup: load %lld compact %lld tables %lld fold %lld fuse %lld | batches %lld (nb %d, ops %d)\n",
