@@ -159,6 +159,20 @@ mpcgs_status mpcgs_init_phylip(const char* path, const mpcgs_config* cfg, double
  * returns after the work is complete. */
 mpcgs_status mpcgs_sample(mpcgs_ctx* ctx, int32_t n_proposals, int64_t n_samples, uint64_t seed);
 
+/* Checkpoint / resume (long chains): run only steps [first_step, last_step)
+ * of the run mpcgs_sample(n_proposals, n_samples, seed) would do (burn-in +
+ * ceil(n_samples / n_proposals) steps; last_step < 0 -> to its end).  Every random
+ * number is keyed by (seed, global step index) (S21), so a run split at any step
+ * boundary is the same chain, bit for bit (tested).  A checkpoint after step k is the
+ * chain state (mpcgs_save_state), the samples (mpcgs_get_samples: the first
+ * min(max(0, (k - burnin) * N), M) of them), seed, N, M and k; to resume, a context
+ * with the same alignment and configuration takes mpcgs_load_state,
+ * mpcgs_put_samples, then mpcgs_sample_steps(N, M, seed, k, -1).  first_step > 0
+ * with fewer samples stored than the earlier steps drew -> MPCGS_E_STATE; first_step
+ * outside [0, last_step] -> MPCGS_E_ARG. */
+mpcgs_status mpcgs_sample_steps(mpcgs_ctx* ctx, int32_t n_proposals, int64_t n_samples, uint64_t seed,
+                                int64_t first_step, int64_t last_step);
+
 /* theta-hat = argmax L(theta) over the stored samples (Eq. 25-26; S20): a log-spaced
  * grid of n_grid points (3..MPCGS_MAX_GRID) over [S_min, S_max]/(n-1) evaluated on
  * the device, then safeguarded Newton on d lnL/d theta inside the grid cells of every
@@ -178,6 +192,19 @@ mpcgs_status mpcgs_score_trees(mpcgs_ctx* ctx, int32_t n_trees, const int32_t* p
 
 /* Replace the chain state (generator) by a host tree; its logL is recomputed. */
 mpcgs_status mpcgs_set_state(mpcgs_ctx* ctx, const int32_t* parent, const double* age);
+
+/* Checkpoint of the chain state: the generator exactly as the device holds
+ * it -- tree arrays, the branch factors and the cached ln P(D|G) and S_G -- plus
+ * theta0, behind a header naming the alignment shape and configuration.  The caller
+ * owns the host buffer (mpcgs_state_bytes bytes; smaller -> MPCGS_E_ARG).  load_state
+ * rejects a blob of another alignment shape / model / precision (MPCGS_E_ARG), sets
+ * theta0 and, with incremental rescoring, recomputes the generator's partials.
+ * With mpcgs_get_samples / mpcgs_put_samples and mpcgs_sample_steps this resumes a
+ * chain bit for bit (set_state would recompute S_G and the branch factors on the
+ * host, which may differ from the device's in the last bit). */
+size_t mpcgs_state_bytes(const mpcgs_ctx* ctx);
+mpcgs_status mpcgs_save_state(mpcgs_ctx* ctx, void* buf, size_t bytes);
+mpcgs_status mpcgs_load_state(mpcgs_ctx* ctx, const void* buf, size_t bytes);
 
 /* Read the generator: host parent/age [2n-1]; logL and S (nullable). */
 mpcgs_status mpcgs_get_state(mpcgs_ctx* ctx, int32_t* parent, double* age, double* logL,
@@ -216,6 +243,12 @@ mpcgs_status mpcgs_get_samples(mpcgs_ctx* ctx, int64_t first, int64_t count, dou
  * mpcgs_estimate_theta on prescribed sample sets (e.g. S20's bimodal case). */
 mpcgs_status mpcgs_load_samples(mpcgs_ctx* ctx, int64_t count, const double* S, const double* logL,
                                 double theta0);
+/* Restore the sample store of a checkpoint: host S, logL [count] (required when
+ * count > 0), step [count] and slot [count] (nullable -> -1).  0 <= count <=
+ * max_samples else MPCGS_E_ARG.  The samples count as drawn under the context's
+ * current theta0. */
+mpcgs_status mpcgs_put_samples(mpcgs_ctx* ctx, int64_t count, const double* S, const double* logL,
+                               const int64_t* step, const int32_t* slot);
 int64_t mpcgs_num_samples(const mpcgs_ctx* ctx);
 /* Sites the kernels score: distinct columns with compress_patterns, else n_sites. */
 int32_t mpcgs_num_patterns(const mpcgs_ctx* ctx);

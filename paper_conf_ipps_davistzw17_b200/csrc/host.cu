@@ -97,6 +97,7 @@ struct mpcgs_ctx {
         cudaEvent_t end = nullptr;
         int N = 0;
         int64_t M = 0;
+        int64_t stored = 0;  // samples in the store once the loop's last step is done
     } pend;
 };
 
@@ -1412,7 +1413,19 @@ namespace {
 // it); sample_end waits for it.  Loops of several contexts (loci) overlap on the
 // device when they are all begun before any is ended.
 mpcgs_status sample_end(mpcgs_ctx* c);
-mpcgs_status sample_begin(mpcgs_ctx* c, int32_t N, int64_t M, uint64_t seed) {
+// samples stored by the first `k` steps of a run (burn-in draws are not stored; then N
+// per step, the last step fewer: Alg. 1, S17)
+int64_t stored_after(const mpcgs_ctx* c, int32_t N, int64_t M, int64_t k) {
+    const int64_t m = (k - (int64_t)c->burnin) * (int64_t)N;
+    return m < 0 ? 0 : (m > M ? M : m);
+}
+
+// steps [first, last) of the run (burn-in + ceil(M/N) steps; last < 0 -> to the end).
+// first > 0 continues a checkpointed run: the generator (mpcgs_set_state) and the
+// samples of steps [0, first) (mpcgs_put_samples) must be in place -- every random
+// number is keyed by the global step index, so the continuation is the same chain.
+mpcgs_status sample_begin(mpcgs_ctx* c, int32_t N, int64_t M, uint64_t seed, int64_t first = 0,
+                          int64_t last = -1) {
     CHECK_CTX(c);
     if (c->pend.active) return fail(c, MPCGS_E_STATE, "a sampling loop is still pending");
     if (N < 1 || N > c->Nmax || N % c->world != 0 || M < 0 || M > c->Mmax)
@@ -1420,10 +1433,22 @@ mpcgs_status sample_begin(mpcgs_ctx* c, int32_t N, int64_t M, uint64_t seed) {
     if (c->world > 1 && !c->comm)
         return fail(c, MPCGS_E_STATE, "world > 1 without an NCCL id: drive steps with mpcgs_step_local, "
                                       "mpcgs_get_records/put_records and mpcgs_step_finish");
-    const int64_t steps = (int64_t)c->burnin + (M + N - 1) / N;
+    const int64_t total = (int64_t)c->burnin + (M + N - 1) / N;
+    if (last < 0 || last > total) last = total;
+    if (first < 0 || first > last) return fail(c, MPCGS_E_ARG, "step range: 0 <= first <= last");
+    const int64_t stored0 = stored_after(c, N, M, first);
+    if (first > 0 && c->nsamples < stored0)
+        return fail(c, MPCGS_E_STATE, "continuing at this step needs the samples of the earlier steps "
+                                      "in the store (mpcgs_put_samples)");
+    const int64_t steps = total;      // the run's length (k_draw prepares no context past it)
+    const int64_t nrun = last - first;  // steps this call runs
     mpcgs_status st = enter(c);
     if (st) return st;
     CU(cudaMemsetAsync(c->s.counters, 0, 8 * 8, c->work));
+    if (first > 0) {  // counters[0] = step index, counters[1] = samples stored
+        const int64_t cnt[2] = {first, stored0};
+        CU(cudaMemcpyAsync(c->s.counters, cnt, sizeof(cnt), cudaMemcpyHostToDevice, c->work));
+    }
     c->launches = 0;
     c->prune_ms = c->propose_ms = c->draw_ms = 0.0;
     auto one_step = [&]() -> mpcgs_status {
@@ -1438,16 +1463,16 @@ mpcgs_status sample_begin(mpcgs_ctx* c, int32_t N, int64_t M, uint64_t seed) {
         }
         return MPCGS_OK;
     };
-    if ((c->timing & 1) && steps > 0) {
+    if ((c->timing & 1) && nrun > 0) {
         // device-timed steps: events at step boundaries and around every pruning
         // launch; optional L2 flush between steps, outside the timed intervals
-        const size_t need = (size_t)4 * steps;
+        const size_t need = (size_t)4 * nrun;
         while (c->evpool.size() < need) {
             cudaEvent_t ev;
             CU(cudaEventCreate(&ev));
             c->evpool.push_back(ev);
         }
-        for (int64_t k = 0; k < steps; ++k) {
+        for (int64_t k = 0; k < nrun; ++k) {
             if ((c->timing & 2) && c->flush_buf)
                 CU(cudaMemsetAsync(c->flush_buf, (int)(k & 0xff), (size_t)256 << 20, c->work));
             CU(cudaEventRecord(c->evpool[4 * k + 0], c->work));
@@ -1465,9 +1490,9 @@ mpcgs_status sample_begin(mpcgs_ctx* c, int32_t N, int64_t M, uint64_t seed) {
             }
             CU(cudaEventRecord(c->evpool[4 * k + 3], c->work));
         }
-        CU(cudaEventSynchronize(c->evpool[4 * (steps - 1) + 3]));
+        CU(cudaEventSynchronize(c->evpool[4 * (nrun - 1) + 3]));
         double tot = 0.0, pr = 0.0, pp = 0.0, dr = 0.0;
-        for (int64_t k = 0; k < steps; ++k) {
+        for (int64_t k = 0; k < nrun; ++k) {
             float t = 0.f, q = 0.f, p0 = 0.f, d0 = 0.f;
             CU(cudaEventElapsedTime(&t, c->evpool[4 * k + 0], c->evpool[4 * k + 3]));
             CU(cudaEventElapsedTime(&p0, c->evpool[4 * k + 0], c->evpool[4 * k + 1]));
@@ -1485,10 +1510,10 @@ mpcgs_status sample_begin(mpcgs_ctx* c, int32_t N, int64_t M, uint64_t seed) {
     } else {
         // CUDA graph of up to graph_steps steps, replayed; the kernels read the step
         // counter from device memory, so one graph serves every step
-        const int64_t G = std::min<int64_t>(c->graph_steps, std::max<int64_t>(steps, 1));
+        const int64_t G = std::min<int64_t>(c->graph_steps, std::max<int64_t>(nrun, 1));
         cudaGraph_t graph = nullptr;
         cudaGraphExec_t exec = nullptr;
-        const int64_t reps = steps / G, rest = steps % G;
+        const int64_t reps = nrun / G, rest = nrun % G;
         CU(cudaEventRecord(c->ev_b, c->work));
         CU(launch_context(c->s, seed, -1, c->work));  // the first context; later ones come from k_draw
         c->launches = 1;
@@ -1522,6 +1547,7 @@ mpcgs_status sample_begin(mpcgs_ctx* c, int32_t N, int64_t M, uint64_t seed) {
     c->pend.active = true;
     c->pend.N = N;
     c->pend.M = M;
+    c->pend.stored = stored_after(c, N, M, last);
     return MPCGS_OK;
 }
 
@@ -1545,7 +1571,7 @@ mpcgs_status sample_end(mpcgs_ctx* c) {
         c->loop_ms = ms;
     }
     if ((st = check_status(c))) return st;
-    c->nsamples = c->pend.M;
+    c->nsamples = c->pend.stored;
     c->lastN = c->pend.N;
     c->sample_theta0 = c->s.theta0;
     return MPCGS_OK;
@@ -1557,6 +1583,14 @@ extern "C" {
 mpcgs_status mpcgs_sample(mpcgs_ctx* c, int32_t N, int64_t M, uint64_t seed) {
     NvtxRange nvtx_("mpcgs_sample");
     mpcgs_status st = sample_begin(c, N, M, seed);
+    if (st) return st;
+    return sample_end(c);
+}
+
+mpcgs_status mpcgs_sample_steps(mpcgs_ctx* c, int32_t N, int64_t M, uint64_t seed, int64_t first_step,
+                                int64_t last_step) {
+    NvtxRange nvtx_("mpcgs_sample_steps");
+    mpcgs_status st = sample_begin(c, N, M, seed, first_step, last_step);
     if (st) return st;
     return sample_end(c);
 }
@@ -1634,6 +1668,28 @@ mpcgs_status mpcgs_load_samples(mpcgs_ctx* c, int64_t count, const double* S, co
     return MPCGS_OK;
 }
 
+mpcgs_status mpcgs_put_samples(mpcgs_ctx* c, int64_t count, const double* S, const double* logL,
+                               const int64_t* step, const int32_t* slot) {
+    CHECK_CTX(c);
+    if (c->pend.active) return fail(c, MPCGS_E_STATE, "a sampling loop is still pending");
+    if (count < 0 || count > c->Mmax || (count > 0 && (!S || !logL)))
+        return fail(c, MPCGS_E_ARG, "put_samples: 0 <= count <= max_samples, S and logL given");
+    mpcgs_status st = enter(c);
+    if (st) return st;
+    if (count > 0) {
+        CU(cudaMemcpyAsync(c->s.sS, S, 8 * (size_t)count, cudaMemcpyHostToDevice, c->work));
+        CU(cudaMemcpyAsync(c->s.sL, logL, 8 * (size_t)count, cudaMemcpyHostToDevice, c->work));
+        if (step) CU(cudaMemcpyAsync(c->s.sStep, step, 8 * (size_t)count, cudaMemcpyHostToDevice, c->work));
+        else CU(cudaMemsetAsync(c->s.sStep, 0xff, 8 * (size_t)count, c->work));
+        if (slot) CU(cudaMemcpyAsync(c->s.sSlot, slot, 4 * (size_t)count, cudaMemcpyHostToDevice, c->work));
+        else CU(cudaMemsetAsync(c->s.sSlot, 0xff, 4 * (size_t)count, c->work));
+    }
+    if ((st = leave(c))) return st;
+    c->nsamples = count;
+    c->sample_theta0 = c->s.theta0;
+    return MPCGS_OK;
+}
+
 mpcgs_status mpcgs_score_trees(mpcgs_ctx* c, int32_t n_trees, const int32_t* parent, const double* age,
                                double* logL_out) {
     NvtxRange nvtx_("mpcgs_score_trees");
@@ -1655,6 +1711,101 @@ mpcgs_status mpcgs_set_state(mpcgs_ctx* c, const int32_t* parent, const double* 
     mpcgs_status st = enter(c);
     if (st) return st;
     return upload_state(c, parent, age);
+}
+
+// checkpoint blob of the chain state: header, then the device generator arrays as
+// they are (so a restored chain continues bit for bit: the cached ln P(D|G) and S_G and
+// the branch factors the device computed, not host recomputations)
+struct StateHeader {
+    uint32_t magic, version;
+    int32_t n, L_orig, model, precision;
+    double theta0;
+};
+constexpr uint32_t STATE_MAGIC = 0x4b43504du;  // "MPCK"
+
+size_t mpcgs_state_bytes(const mpcgs_ctx* c) {
+    return c ? sizeof(StateHeader) + (size_t)c->nn * (4 * 4 + 3 * 8) + 2 * 8 : 0;
+}
+
+mpcgs_status mpcgs_save_state(mpcgs_ctx* c, void* buf, size_t bytes) {
+    CHECK_CTX(c);
+    if (!buf || bytes < mpcgs_state_bytes(c)) return fail(c, MPCGS_E_ARG, "save_state: buffer too small");
+    mpcgs_status st = enter(c);
+    if (st) return st;
+    const size_t nn = (size_t)c->nn;
+    StateHeader h{STATE_MAGIC, 1u, c->n, c->L_orig, c->model, c->precision, c->s.theta0};
+    unsigned char* p = static_cast<unsigned char*>(buf);
+    std::memcpy(p, &h, sizeof(h));
+    p += sizeof(h);
+    for (int32_t* a : {c->s.parent, c->s.left, c->s.right, c->s.need}) {
+        CU(cudaMemcpyAsync(p, a, 4 * nn, cudaMemcpyDeviceToHost, c->work));
+        p += 4 * nn;
+    }
+    for (double* a : {c->s.age, c->s.e, c->s.em}) {
+        CU(cudaMemcpyAsync(p, a, 8 * nn, cudaMemcpyDeviceToHost, c->work));
+        p += 8 * nn;
+    }
+    CU(cudaMemcpyAsync(p, c->s.gen, 16, cudaMemcpyDeviceToHost, c->work));
+    return leave(c);
+}
+
+mpcgs_status mpcgs_load_state(mpcgs_ctx* c, const void* buf, size_t bytes) {
+    CHECK_CTX(c);
+    if (c->pend.active) return fail(c, MPCGS_E_STATE, "a sampling loop is still pending");
+    if (!buf || bytes < mpcgs_state_bytes(c)) return fail(c, MPCGS_E_ARG, "load_state: buffer too small");
+    StateHeader h;
+    std::memcpy(&h, buf, sizeof(h));
+    if (h.magic != STATE_MAGIC || h.version != 1u || h.n != c->n || h.L_orig != c->L_orig || h.model != c->model ||
+        h.precision != c->precision || !(h.theta0 > 0.0))
+        return fail(c, MPCGS_E_ARG, "load_state: not a checkpoint of this alignment / configuration");
+    const size_t nn = (size_t)c->nn;
+    const unsigned char* p = static_cast<const unsigned char*>(buf) + sizeof(h);
+    std::vector<int32_t> parent(nn), left(nn), right(nn);
+    std::memcpy(parent.data(), p, 4 * nn);
+    std::memcpy(left.data(), p + 4 * nn, 4 * nn);
+    std::memcpy(right.data(), p + 8 * nn, 4 * nn);
+    std::vector<double> age(nn);
+    std::memcpy(age.data(), p + 16 * nn, 8 * nn);
+    std::string why;
+    if (check_tree(c->n, parent.data(), age.data(), why)) return fail(c, MPCGS_E_ARG, "load_state: " + why);
+    mpcgs_status st = enter(c);
+    if (st) return st;
+    for (int32_t* a : {c->s.parent, c->s.left, c->s.right, c->s.need}) {
+        CU(cudaMemcpyAsync(a, p, 4 * nn, cudaMemcpyHostToDevice, c->work));
+        p += 4 * nn;
+    }
+    for (double* a : {c->s.age, c->s.e, c->s.em}) {
+        CU(cudaMemcpyAsync(a, p, 8 * nn, cudaMemcpyHostToDevice, c->work));
+        p += 8 * nn;
+    }
+    CU(cudaMemcpyAsync(c->s.gen, p, 16, cudaMemcpyHostToDevice, c->work));
+    c->theta0 = h.theta0;
+    c->s.theta0 = h.theta0;
+    if (c->incremental) {  // the generator's stored partials (interior nodes children-first)
+        const int n = c->n;
+        int root = 0;
+        for (size_t v = 0; v < nn; ++v)
+            if (parent[v] < 0) root = (int)v;
+        std::vector<int32_t> order;
+        std::vector<int> stk{root};
+        std::vector<char> done(nn, 0);
+        while (!stk.empty()) {
+            const int v = stk.back();
+            const int a = left[v], b2 = right[v];
+            if ((a >= n && !done[a]) || (b2 >= n && !done[b2])) {
+                if (a >= n && !done[a]) stk.push_back(a);
+                if (b2 >= n && !done[b2]) stk.push_back(b2);
+                continue;
+            }
+            done[v] = 1;
+            order.push_back(v);
+            stk.pop_back();
+        }
+        CU(cudaMemcpyAsync(c->s.gen_order, order.data(), 4 * order.size(), cudaMemcpyHostToDevice, c->work));
+        CU(launch_gen_partials(c->s, c->work));
+    }
+    CU(cudaStreamSynchronize(c->work));
+    return leave(c);
 }
 
 mpcgs_status mpcgs_get_state(mpcgs_ctx* c, int32_t* parent, double* age, double* logL, double* S) {

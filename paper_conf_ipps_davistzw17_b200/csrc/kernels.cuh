@@ -39,6 +39,7 @@ struct PruneArgs {
     const int32_t* tree_need;  // [ntrees] register need of each tree's schedule (nullable)
     int need_cap;              // set by launch_prune: largest need the table kernel serves
     int trip_cap;              // set by launch_prune: fused triplets per tree (table kernel)
+    int code_bufs;             // set by launch_prune: tip-code staging buffers of the table kernel (1 or 2)
     int unit_batches;          // table kernel: site batches per exact-sum unit (tiles hold whole units)
     unsigned long long* tree_acc;  // [ntrees][4] exact site-sum accumulators (Exact128), zero on entry
     uint32_t* tile_cnt;        // [ntrees], zero on entry, reset by the kernel

@@ -51,16 +51,27 @@ int prune_need_cap(int n) { return std::min(prune_max_need(n), PRUNE_DR + (n <= 
 
 
 template <typename T, bool GM>
-static size_t tab_bytes_for(int n, bool amb = false) {
+static size_t tab_bytes_for(int n, bool amb = false, int bufs = 2) {
     const int cap = prune_need_cap(n);
     constexpr int SI = sizeof(T) == 4 ? PRUNE_SI32 : PRUNE_SI64;
     if (amb)  // 4-bit base-set codes, 16-row tip tables (S24)
-        return wide_sites(n) ? tab_smem_bytes<T, PRUNE_DR, SI, false, GM, 4>(n - 1, cap, 0)
-                             : tab_smem_bytes<T, PRUNE_DR, PRUNE_SI_LARGE, false, GM, 4>(n - 1, cap, 0);
+        return wide_sites(n) ? tab_smem_bytes<T, PRUNE_DR, SI, false, GM, 4>(n - 1, cap, 0, bufs)
+                             : tab_smem_bytes<T, PRUNE_DR, PRUNE_SI_LARGE, false, GM, 4>(n - 1, cap, 0, bufs);
     const bool pt = product_tables<T, GM>(n);
-    if (pt && !wide_sites(n)) return tab_smem_bytes<T, PRUNE_DR, PRUNE_SI_LARGE, true, GM>(n - 1, cap, 0);
-    return pt ? tab_smem_bytes<T, PRUNE_DR, SI, true, GM>(n - 1, cap, 0)
-                             : tab_smem_bytes<T, PRUNE_DR, PRUNE_SI_LARGE, false, GM>(n - 1, cap, 0);
+    if (pt && !wide_sites(n)) return tab_smem_bytes<T, PRUNE_DR, PRUNE_SI_LARGE, true, GM>(n - 1, cap, 0, bufs);
+    return pt ? tab_smem_bytes<T, PRUNE_DR, SI, true, GM>(n - 1, cap, 0, bufs)
+              : tab_smem_bytes<T, PRUNE_DR, PRUNE_SI_LARGE, false, GM>(n - 1, cap, 0, bufs);
+}
+
+// resident CTAs per SM the shared memory of `bytes` allows (228 KB per SM, 1 KB reserved per CTA)
+static int by_smem(size_t bytes) { return (int)((228 * 1024) / (bytes + 1024 + 256)); }
+
+// the layout launch_tab_w picks: one code buffer when that buys a resident CTA
+template <typename T, bool GM>
+static size_t tab_bytes_best(int n, bool amb = false) {
+    const int regcap = sizeof(T) == 4 ? 4 : 3;
+    const size_t b2 = tab_bytes_for<T, GM>(n, amb, 2), b1 = tab_bytes_for<T, GM>(n, amb, 1);
+    return (MPCGS_SINGLEBUF && std::min(regcap, by_smem(b1)) > std::min(regcap, by_smem(b2))) ? b1 : b2;
 }
 
 #ifndef MPCGS_TAB_MIN_N
@@ -70,17 +81,16 @@ static size_t tab_bytes_for(int n, bool amb = false) {
 // (159 registers FP64 -> 3, FP32 -> 4) or the shared-memory limit of the base layout
 int prune_resident_per_sm(int n, int precision, bool general_model) {
     size_t bytes;
-    if (precision == 32) bytes = general_model ? tab_bytes_for<float, true>(n) : tab_bytes_for<float, false>(n);
-    else bytes = general_model ? tab_bytes_for<double, true>(n) : tab_bytes_for<double, false>(n);
-    const int by_smem = (int)((228 * 1024) / (bytes + 1024 + 256));
-    return std::max(1, std::min(precision == 32 ? 4 : 3, by_smem));
+    if (precision == 32) bytes = general_model ? tab_bytes_best<float, true>(n) : tab_bytes_best<float, false>(n);
+    else bytes = general_model ? tab_bytes_best<double, true>(n) : tab_bytes_best<double, false>(n);
+    return std::max(1, std::min(precision == 32 ? 4 : 3, by_smem(bytes)));
 }
 
 bool prune_uses_tables(int n, int precision, bool general_model, bool amb) {
     if (n < MPCGS_TAB_MIN_N) return false;
     size_t bytes;
-    if (precision == 32) bytes = general_model ? tab_bytes_for<float, true>(n, amb) : tab_bytes_for<float, false>(n, amb);
-    else bytes = general_model ? tab_bytes_for<double, true>(n, amb) : tab_bytes_for<double, false>(n, amb);
+    if (precision == 32) bytes = general_model ? tab_bytes_best<float, true>(n, amb) : tab_bytes_best<float, false>(n, amb);
+    else bytes = general_model ? tab_bytes_best<double, true>(n, amb) : tab_bytes_best<double, false>(n, amb);
     return bytes <= 160 * 1024;
 }
 

@@ -842,19 +842,60 @@ __device__ __forceinline__ void run_op(int di, Stack<T, DR, SI>& st, uint32_t co
 
 __host__ __device__ constexpr size_t align16(size_t x) { return (x + 15) & ~(size_t)15; }
 
-// shared memory of the table kernel for trees of n tips whose register need is
-// at most `need` (spill levels above DR), with up to `trip_cap` fused triplets
+// Shared-memory layout of the table kernel for trees of n tips whose register need is
+// at most `need` (spill levels above DR), with up to `trip_cap` fused triplets and
+// `bufs` tip-code staging buffers.  F81: the per-op branch data s_e and the setup
+// arrays s_d / s_tl are dead once the op loop starts, so they live in space the loop
+// only needs later -- the second code buffer (double buffering: first filled by the
+// prefetch of batch 1, after the setup) or the shared spill levels (single buffer).
+// bufs = 1 is chosen where it buys a resident CTA per SM (n = 256: 2 -> 3).
+#ifndef MPCGS_ALIAS
+#define MPCGS_ALIAS 1
+#endif
+#ifndef MPCGS_SINGLEBUF
+#define MPCGS_SINGLEBUF 1
+#endif
 template <typename T, int DR, int SI, bool PT, bool GM = false, int BITS = 2>
-__host__ __device__ size_t tab_smem_bytes(int nops, int need, int trip_cap) {
-    const int n = nops + 1;
-    const int spill = need > DR ? need - DR : 0;
-    return align16(GM ? 2 * GMC * sizeof(T) * nops + GMC * sizeof(T) : sizeof(typename Traits<T>::E4) * nops) +
-           align16(sizeof(T) * ((PT ? 32 : (BITS == 4 ? 64 : 16)) * (size_t)n + (size_t)TRIP_EXTRA * (PT ? trip_cap : 0))) +
-           align16(sizeof(OpRec<T>) * nops) + 2 * align16(Codes<SI, BITS>::buf_bytes(n)) +
-           sizeof(T) * (size_t)spill * SI * 4 * PRUNE_THREADS +
-           align16(sizeof(int) * 2 * (size_t)nops) + align16(sizeof(int) * (size_t)nops) +
-           (GM && sizeof(T) == 8 && BITS == 2 ? align16(sizeof(int) * (size_t)(nops + 1)) : 0) +  // slot rows
-           64 * sizeof(int);
+struct TabLayout {
+    size_t e, tab, opc, cod, bufb, spill, d, tl, pos, total;
+    __host__ __device__ TabLayout(int nops, int need, int trip_cap, int bufs) {
+        const int n = nops + 1;
+        const size_t e_bytes = align16(GM ? 2 * GMC * sizeof(T) * nops + GMC * sizeof(T)
+                                          : sizeof(typename Traits<T>::E4) * nops);
+        const size_t d_bytes = align16(sizeof(int) * 2 * (size_t)nops), tl_bytes = align16(sizeof(int) * (size_t)nops);
+        const size_t spill_bytes = sizeof(T) * (size_t)(need > DR ? need - DR : 0) * SI * 4 * PRUNE_THREADS;
+        const size_t scratch = e_bytes + d_bytes + tl_bytes;
+        bufb = align16(Codes<SI, BITS>::buf_bytes(n));
+        const bool in_buf1 = MPCGS_ALIAS && !GM && bufs == 2 && scratch <= bufb;
+        const bool in_spill = MPCGS_ALIAS && !GM && !in_buf1 && scratch <= spill_bytes;
+        size_t o = 0;
+        e = 0;
+        if (!in_buf1 && !in_spill) o += e_bytes;
+        tab = o;
+        o += align16(sizeof(T) * ((PT ? 32 : (BITS == 4 ? 64 : 16)) * (size_t)n + (size_t)TRIP_EXTRA * (PT ? trip_cap : 0)));
+        opc = o;
+        o += align16(sizeof(OpRec<T>) * nops);
+        cod = o;
+        o += (size_t)bufs * bufb;
+        spill = o;
+        o += spill_bytes;
+        if (in_buf1 || in_spill) {
+            e = in_buf1 ? cod + bufb : spill;
+            d = e + e_bytes;
+            tl = d + d_bytes;
+        } else {
+            d = o;
+            tl = d + d_bytes;
+            o = tl + tl_bytes;
+        }
+        pos = o;  // tip -> code row (slot_rows only)
+        if (GM && sizeof(T) == 8 && BITS == 2) o += align16(sizeof(int) * (size_t)(nops + 1));
+        total = o + 64 * sizeof(int);
+    }
+};
+template <typename T, int DR, int SI, bool PT, bool GM = false, int BITS = 2>
+__host__ __device__ size_t tab_smem_bytes(int nops, int need, int trip_cap, int bufs = 2) {
+    return TabLayout<T, DR, SI, PT, GM, BITS>(nops, need, trip_cap, bufs).total;
 }
 
 #ifdef MPCGS_MINB  // tuning builds only: min CTAs per SM (caps registers)
@@ -887,23 +928,22 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
     constexpr size_t OPB = GM ? 2 * GMC * sizeof(T) : sizeof(E4);  // branch data bytes per op
     const int nops = a.nops, n = nops + 1;
     const int trip_cap = PT ? a.trip_cap : 0;
-    E4* s_e = reinterpret_cast<E4*>(smem_raw);  // F81: {e_a, em_a, e_b, em_b} per op
-    T* s_P = reinterpret_cast<T*>(smem_raw);    // general model: branch records {C_a, C_b} per op
+    const int bufs = a.code_bufs == 1 ? 1 : 2;
+    const TabLayout<T, DR, SI, PT, GM, BITS> lay(nops, a.need_cap, trip_cap, bufs);
+    E4* s_e = reinterpret_cast<E4*>(smem_raw + lay.e);  // F81: {e_a, em_a, e_b, em_b} per op
+    T* s_P = reinterpret_cast<T*>(smem_raw + lay.e);    // general model: branch records {C_a, C_b} per op
     // general model: {C_a, C_b} of every op, then the identity record (the root's up branch)
-    T* s_tab = reinterpret_cast<T*>(smem_raw + align16(OPB * nops + (GM ? GMC * sizeof(T) : 0)));
+    T* s_tab = reinterpret_cast<T*>(smem_raw + lay.tab);
     // compacted ops: {code, table byte offset, original op index, tip c of a fused triplet}
-    OpRec<T>* s_opc = reinterpret_cast<OpRec<T>*>(reinterpret_cast<unsigned char*>(s_tab) +
-                                            align16(sizeof(T) * (TABE * n + (size_t)TRIP_EXTRA * trip_cap)));
-    unsigned char* s_cod = reinterpret_cast<unsigned char*>(s_opc) + align16(sizeof(OpRec<T>) * nops);
-    const size_t bufb = align16(CD::buf_bytes(n));
-    T* s_spill = reinterpret_cast<T*>(s_cod + 2 * bufb);
-    const int spill_lv = a.need_cap > DR ? a.need_cap - DR : 0;
-    int* s_d = reinterpret_cast<int*>(reinterpret_cast<unsigned char*>(s_spill) +
-                                      sizeof(T) * (size_t)spill_lv * SI * 4 * PRUNE_THREADS);
-    int* s_tl = s_d + align16(sizeof(int) * 2 * (size_t)nops) / sizeof(int);  // original codes, then check flags
+    OpRec<T>* s_opc = reinterpret_cast<OpRec<T>*>(smem_raw + lay.opc);
+    unsigned char* s_cod = smem_raw + lay.cod;
+    const size_t bufb = lay.bufb;
+    T* s_spill = reinterpret_cast<T*>(smem_raw + lay.spill);
+    int* s_d = reinterpret_cast<int*>(smem_raw + lay.d);
+    int* s_tl = reinterpret_cast<int*>(smem_raw + lay.tl);  // original codes, then check flags
     // tip -> code row (slot_rows only: reserved for FP64 general-model 2-bit kernels; every
     // byte here costs the others triplet tables, FP32 c5 -3.8 % with it)
-    int* s_pos = s_tl + align16(sizeof(int) * (size_t)nops) / sizeof(int);
+    int* s_pos = reinterpret_cast<int*>(smem_raw + lay.pos);
     __shared__ int s_nc;  // compacted op count
 
     const int tid = threadIdx.x;
@@ -1294,14 +1334,14 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
     for (int b0 = 0; b0 < nb; b0 += a.unit_batches) {
         const int b1 = min(nb, b0 + a.unit_batches);
         for (int b = b0; b < b1; ++b) {
-            if (b + 1 < nb) {
+            if (bufs == 2 && b + 1 < nb) {
                 issue(b + 1, (b + 1) & 1);
                 cp_async_wait<1>();
-            } else {
+            } else {  // last batch, or one buffer: this batch's codes were issued before
                 cp_async_wait<0>();
             }
             __syncthreads();
-            cc.sbase = smem_addr(s_cod + (size_t)(b & 1) * bufb);
+            cc.sbase = smem_addr(s_cod + (size_t)(bufs == 2 ? (b & 1) : 0) * bufb);
             int scale[SI];
 #pragma unroll
             for (int k = 0; k < SI; ++k) scale[k] = 0;
@@ -1330,7 +1370,8 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
                 ls = fma(pi[3], root[3], ls);
                 if (site0 + k < s_end) acc.add((double)ls, scale[k], a.site_w, site0 + k);  // padding not counted
             }
-            __syncthreads();  // the buffer of batch b is refilled in iteration b+1
+            __syncthreads();  // the buffer of batch b is refilled in iteration b+1 (one buffer: now)
+            if (bufs == 1 && b + 1 < nb) issue(b + 1, 0);
         }
         // this thread's log over the unit (0 if it had no site there)
         ex.add(acc.total());
@@ -1395,33 +1436,46 @@ static cudaError_t launch_flat(const PruneArgs& a, int ntrees, cudaStream_t st) 
 // bound it), so fusion never costs a resident CTA.  Cached per tree size; the
 // first call is at init (mpcgs_init scores G0), outside any graph capture.
 template <typename T, int DR, int SI, bool PT, bool GM, int BITS, typename K>
-static int tab_trip_cap(K kern, int nops, int need_cap) {
-    if (!PT || MPCGS_NO_TRIPLETS) return 0;
-    static int key[8] = {-1, -1, -1, -1, -1, -1, -1, -1}, val[8];
+static int tab_trip_cap(K kern, int nops, int need_cap, int& bufs) {
+    // one or two tip-code buffers: one when it buys a resident CTA (cached per tree size)
+    static int key[8] = {-1, -1, -1, -1, -1, -1, -1, -1}, val[8], vbufs[8];
     const int k = nops * 16 + need_cap;
     for (int i = 0; i < 8; ++i)
-        if (key[i] == k) return val[i];
-    const size_t base = tab_smem_bytes<T, DR, SI, PT, GM, BITS>(nops, need_cap, 0);
-    int dev = 0, per_sm = 0, resv = 0, optin = 0, blocks = 0;
+        if (key[i] == k) {
+            bufs = vbufs[i];
+            return val[i];
+        }
+    int dev = 0, per_sm = 0, resv = 0, optin = 0, blocks = 0, blocks1 = 0;
     cudaGetDevice(&dev);
     cudaDeviceGetAttribute(&per_sm, cudaDevAttrMaxSharedMemoryPerMultiprocessor, dev);
     cudaDeviceGetAttribute(&resv, cudaDevAttrReservedSharedMemoryPerBlock, dev);
     cudaDeviceGetAttribute(&optin, cudaDevAttrMaxSharedMemoryPerBlockOptin, dev);
     int cap = 0;
+    bufs = 2;
+    size_t base = tab_smem_bytes<T, DR, SI, PT, GM, BITS>(nops, need_cap, 0, 2);
+    const size_t base1 = tab_smem_bytes<T, DR, SI, PT, GM, BITS>(nops, need_cap, 0, 1);
     cudaFuncAttributes fa{};
     if (cudaFuncGetAttributes(&fa, kern) == cudaSuccess &&
         cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, optin - (int)fa.sharedSizeBytes) ==
             cudaSuccess &&
         cudaOccupancyMaxActiveBlocksPerMultiprocessor(&blocks, kern, PRUNE_THREADS, base) == cudaSuccess &&
-        blocks > 0) {
-        const long room = std::min<long>(optin, per_sm / blocks - resv - 256) - (long)fa.sharedSizeBytes - (long)base;
-        cap = (int)std::max<long>(0, std::min<long>((nops + 1) / 3, room / (long)(sizeof(T) * TRIP_EXTRA)));
+        cudaOccupancyMaxActiveBlocksPerMultiprocessor(&blocks1, kern, PRUNE_THREADS, base1) == cudaSuccess) {
+        if (MPCGS_SINGLEBUF && blocks1 > blocks) {
+            bufs = 1;
+            base = base1;
+            blocks = blocks1;
+        }
+        if (PT && !MPCGS_NO_TRIPLETS && blocks > 0) {
+            const long room = std::min<long>(optin, per_sm / blocks - resv - 256) - (long)fa.sharedSizeBytes - (long)base;
+            cap = (int)std::max<long>(0, std::min<long>((nops + 1) / 3, room / (long)(sizeof(T) * TRIP_EXTRA)));
+        }
     }
     cudaGetLastError();
     for (int i = 0; i < 8; ++i)
         if (key[i] < 0) {
             key[i] = k;
             val[i] = cap;
+            vbufs[i] = bufs;
             break;
         }
     return cap;
@@ -1430,8 +1484,8 @@ static int tab_trip_cap(K kern, int nops, int need_cap) {
 template <typename T, int DR, int SI, bool PT, int DMX, bool W, bool GM, int BITS>
 static cudaError_t launch_tab_w(PruneArgs a, int ntrees, cudaStream_t st) {
     auto kern = k_prune_tab<T, DR, SI, PT, DMX, W, GM, BITS>;
-    a.trip_cap = tab_trip_cap<T, DR, SI, PT, GM, BITS>(kern, a.nops, a.need_cap);
-    const size_t smem = tab_smem_bytes<T, DR, SI, PT, GM, BITS>(a.nops, a.need_cap, a.trip_cap);
+    a.trip_cap = tab_trip_cap<T, DR, SI, PT, GM, BITS>(kern, a.nops, a.need_cap, a.code_bufs);
+    const size_t smem = tab_smem_bytes<T, DR, SI, PT, GM, BITS>(a.nops, a.need_cap, a.trip_cap, a.code_bufs);
     static size_t attr_bytes = 48 * 1024;
     if (smem > attr_bytes) {
         cudaError_t e = cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);

@@ -61,6 +61,11 @@ _SIGS = {
     "mpcgs_init": (_i32, [_P, _P, _f64, _P]),
     "mpcgs_init_phylip": (_i32, [ctypes.c_char_p, _P, _f64, _P]),
     "mpcgs_sample": (_i32, [_P, _i32, _i64, _u64]),
+    "mpcgs_sample_steps": (_i32, [_P, _i32, _i64, _u64, _i64, _i64]),
+    "mpcgs_put_samples": (_i32, [_P, _i64, _P, _P, _P, _P]),
+    "mpcgs_state_bytes": (ctypes.c_size_t, [_P]),
+    "mpcgs_save_state": (_i32, [_P, _P, ctypes.c_size_t]),
+    "mpcgs_load_state": (_i32, [_P, _P, ctypes.c_size_t]),
     "mpcgs_estimate_theta": (_i32, [_P, _P, _i32, _P, _P]),
     "mpcgs_log_rel_likelihood": (_i32, [_P, _f64, _P]),
     "mpcgs_score_trees": (_i32, [_P, _i32, _P, _P, _P]),
@@ -377,6 +382,30 @@ class Context:
 
     def mpcgs_sample(self, n_proposals, n_samples, seed):
         self._chk(lib().mpcgs_sample(self.h, n_proposals, n_samples, seed), "sample")
+
+    def mpcgs_sample_steps(self, n_proposals, n_samples, seed, first_step, last_step=-1):
+        """Steps [first_step, last_step) of the mpcgs_sample run (checkpoint / resume)."""
+        self._chk(lib().mpcgs_sample_steps(self.h, n_proposals, n_samples, seed, first_step, last_step),
+                  "sample_steps")
+
+    def mpcgs_save_state(self):
+        """Checkpoint blob of the chain state (bytes)."""
+        nb = lib().mpcgs_state_bytes(self.h)
+        buf = np.zeros(nb, np.uint8)
+        self._chk(lib().mpcgs_save_state(self.h, _ptr(buf), nb), "save_state")
+        return buf.tobytes()
+
+    def mpcgs_load_state(self, blob):
+        buf = np.frombuffer(blob, dtype=np.uint8).copy()
+        self._chk(lib().mpcgs_load_state(self.h, _ptr(buf), buf.size), "load_state")
+
+    def mpcgs_put_samples(self, S, logL, step=None, slot=None):
+        """Restore a checkpoint's sample store (step / slot optional)."""
+        S = _f64a(S)
+        ll = _f64a(logL, S.size)
+        st = None if step is None else np.ascontiguousarray(step, dtype=np.int64)
+        sl = None if slot is None else np.ascontiguousarray(slot, dtype=np.int32)
+        self._chk(lib().mpcgs_put_samples(self.h, S.size, _ptr(S), _ptr(ll), _ptr(st), _ptr(sl)), "put_samples")
 
     def mpcgs_estimate_theta(self, n_grid=256, curve=False):
         th = ctypes.c_double()

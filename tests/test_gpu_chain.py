@@ -134,3 +134,89 @@ def test_em_trace_matches_oracle(P, orc):
         gp, ga, _, _ = ctx.mpcgs_get_state()
         assert np.array_equal(gp, ref["parent"])
         assert np.allclose(ga, ref["age"], rtol=0, atol=1e-10 * ref["age"].max())
+
+
+@pytest.mark.parametrize("split", [5, 20, 41])  # inside burn-in, at its end, mid-sampling
+@pytest.mark.parametrize("timing", [0, 1])
+def test_checkpoint_resume_same_chain(P, orc, split, timing):
+    """Checkpoint / resume: the c2 chain run to step `split`, checkpointed
+    (mpcgs_save_state, samples), and resumed in a fresh context (mpcgs_load_state,
+    mpcgs_put_samples, mpcgs_sample_steps) is the uninterrupted chain bit for bit --
+    samples (S, ln L, step, slot) and the final generator.  Every random number is
+    keyed by (seed, global step) (S21)."""
+    wl, codes, pi, u, parent, age, N, B, M, seed, _ = _setup(orc, "c2")
+    rows = synth.to_strings(codes)
+
+    def fresh():
+        ctx = P.Context(rows, wl["theta0"], init_tree=(parent, age), burnin_steps=B, max_proposals=N,
+                        max_samples=M)
+        ctx.mpcgs_set_timing(timing)
+        return ctx
+
+    full = fresh()
+    full.mpcgs_sample(N, M, seed)
+    want = full.mpcgs_get_samples()
+    want_state = full.mpcgs_get_state()
+
+    first = fresh()
+    first.mpcgs_sample_steps(N, M, seed, 0, split)
+    stored = first.mpcgs_num_samples()
+    assert stored == max(0, min(M, (split - B) * N))
+    blob = first.mpcgs_save_state()
+    ck_state = first.mpcgs_get_state()
+    ck = first.mpcgs_get_samples() if stored else None
+    first.free()
+
+    second = fresh()
+    second.mpcgs_load_state(blob)
+    got_state = second.mpcgs_get_state()
+    for a, b in zip(got_state, ck_state):
+        assert np.array_equal(a, b)
+    if ck is not None:
+        second.mpcgs_put_samples(ck["S"], ck["logL"], ck["step"], ck["slot"])
+    second.mpcgs_sample_steps(N, M, seed, split)
+    assert second.mpcgs_num_samples() == M
+    got = second.mpcgs_get_samples()
+    for k in want:
+        assert np.array_equal(got[k], want[k]), k
+    gs = second.mpcgs_get_state()
+    assert np.array_equal(gs[0], want_state[0]) and np.array_equal(gs[1], want_state[1])
+
+
+def test_set_state_recomputes_cached_likelihood(P, orc):
+    """mpcgs_set_state rescores the given tree: ln P(D|G) is tiling-invariant (P22), so
+    the recomputed value matches the one the chain cached when the tree was scored as
+    one of N proposals -- up to the host's branch factors exp(-u t) (set_state) against
+    the device's (k_propose), which may differ in the last bit."""
+    wl, codes, pi, u, parent, age, N, B, M, seed, _ = _setup(orc, "c2")
+    ctx = P.Context(synth.to_strings(codes), wl["theta0"], init_tree=(parent, age), burnin_steps=B,
+                    max_proposals=N, max_samples=M)
+    ctx.mpcgs_sample_steps(N, M, seed, 0, 30)
+    gp, ga, gl, _ = ctx.mpcgs_get_state()
+    ctx.mpcgs_set_state(gp, ga)
+    assert abs(ctx.mpcgs_get_state()[2] - gl) <= 1e-12 * abs(gl)
+
+
+def test_load_state_rejects_other_configuration(P, orc):
+    wl, codes, pi, u, parent, age, N, B, M, seed, _ = _setup(orc, "c2")
+    rows = synth.to_strings(codes)
+    a = P.Context(rows, wl["theta0"], init_tree=(parent, age), max_proposals=N, max_samples=M)
+    blob = a.mpcgs_save_state()
+    b = P.Context(rows, wl["theta0"], init_tree=(parent, age), max_proposals=N, max_samples=M, precision=32)
+    with pytest.raises(P.MpcgsError):
+        b.mpcgs_load_state(blob)
+    with pytest.raises(P.MpcgsError):
+        a.mpcgs_load_state(blob[:-8])  # truncated
+    a.mpcgs_load_state(blob)
+
+
+def test_sample_steps_argument_errors(P, orc):
+    wl, codes, pi, u, parent, age, N, B, M, seed, _ = _setup(orc, "c2")
+    ctx = P.Context(synth.to_strings(codes), wl["theta0"], init_tree=(parent, age), burnin_steps=B,
+                    max_proposals=N, max_samples=M)
+    with pytest.raises(P.MpcgsError):
+        ctx.mpcgs_sample_steps(N, M, seed, 30, 10)  # first > last
+    with pytest.raises(P.MpcgsError):
+        ctx.mpcgs_sample_steps(N, M, seed, 30)      # the samples of steps 20..29 are missing
+    ctx.mpcgs_sample_steps(N, M, seed, 0, 10)       # burn-in only: nothing stored
+    assert ctx.mpcgs_num_samples() == 0

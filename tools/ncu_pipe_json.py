@@ -52,6 +52,10 @@ entry = {
     "fp64_thread_inst_per_partial": fp64 / partials if fp64 else None,
     "fp32_thread_inst_per_partial": fp32 / partials if fp32 else None,
     "shared_bank_conflicts": f("l1tex__data_bank_conflicts_pipe_lsu_mem_shared.sum"),
+    "shared_wavefronts": f("l1tex__data_pipe_lsu_wavefronts_mem_shared.sum"),
+    # one shared-memory wavefront per SM per cycle at most
+    "shared_wavefront_pct": 100.0 * f("l1tex__data_pipe_lsu_wavefronts_mem_shared.sum") /
+                            max(1.0, f("sm__cycles_elapsed.avg") * f("device__attribute_multiprocessor_count")),
     "dram_bytes": nbytes("dram__bytes_read.sum") + nbytes("dram__bytes_write.sum"),
     "source": note,
 }

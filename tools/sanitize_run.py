@@ -38,4 +38,22 @@ for ck in r:
     ck.mpcgs_step_finish(0, 64, 64, 9)
 c.mpcgs_load_samples(np.array([1.0, 100.0, 3.0]), 2.15)
 print("bimodal theta-hat", c.mpcgs_estimate_theta(64))
+# n = 256 (single code buffer, setup arrays aliased into the spill levels), F81 and HKY85
+for model, kappa in (("F81", 0.0), ("HKY85", 4.0)):
+    wl = synth.workload("c4", n=256, L=600, N=4)
+    c = P.Context(synth.to_strings(wl["codes"]), wl["theta0"], init_tree=(wl["true_parent"], wl["true_age"]),
+                  model=model, kappa=kappa, burnin_steps=1, max_proposals=4, max_samples=8)
+    c.mpcgs_sample(4, 8, 11)
+    print("n=256", model, c.mpcgs_get_samples()["logL"][:2])
+# checkpoint / resume
+wl = synth.workload("c2", L=300)
+rows = synth.to_strings(wl["codes"])
+a = P.Context(rows, wl["theta0"], burnin_steps=2, max_proposals=16, max_samples=64)
+a.mpcgs_sample_steps(16, 64, 3, 0, 4)
+blob, smp = a.mpcgs_save_state(), a.mpcgs_get_samples()
+b = P.Context(rows, wl["theta0"], burnin_steps=2, max_proposals=16, max_samples=64)
+b.mpcgs_load_state(blob)
+b.mpcgs_put_samples(smp["S"], smp["logL"], smp["step"], smp["slot"])
+b.mpcgs_sample_steps(16, 64, 3, 4)
+print("resumed", b.mpcgs_num_samples())
 print("sanitize run done")
