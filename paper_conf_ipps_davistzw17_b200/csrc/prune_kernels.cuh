@@ -1465,6 +1465,9 @@ static int tab_trip_cap(K kern, int nops, int need_cap, int& bufs) {
             base = base1;
             blocks = blocks1;
         }
+#ifdef MPCGS_GM32_MAXCTA  // tuning: occupancy cap of the FP32 general-model kernel (room for triplets)
+        if (GM && sizeof(T) == 4) blocks = std::min(blocks, MPCGS_GM32_MAXCTA);
+#endif
         if (PT && !MPCGS_NO_TRIPLETS && blocks > 0) {
             const long room = std::min<long>(optin, per_sm / blocks - resv - 256) - (long)fa.sharedSizeBytes - (long)base;
             cap = (int)std::max<long>(0, std::min<long>((nops + 1) / 3, room / (long)(sizeof(T) * TRIP_EXTRA)));
@@ -1504,11 +1507,16 @@ static cudaError_t launch_tab(const PruneArgs& a, int ntrees, cudaStream_t st) {
 }
 
 constexpr int PRUNE_SI_LARGE = 2;  // sites per thread for n > 128
-inline bool wide_sites(int n) { return n <= 128; }  // SI sites per thread (else PRUNE_SI_LARGE)
+#ifndef MPCGS_WIDE_MAX
+#define MPCGS_WIDE_MAX 128
+#endif
+inline bool wide_sites(int n) { return n <= MPCGS_WIDE_MAX; }  // SI sites per thread (else PRUNE_SI_LARGE)
 // cherry (16x4) / fused-triplet (64x4) tables: always up to 128 tips; above (with 2 sites
-// per thread) only while their shared memory still leaves two CTAs per SM (measured:
-// FP64 n = 192 +12 %, FP32 n = 256 +43 %; FP64 n = 256 needs one CTA per SM and is 20 %
-// slower with tables than without)
+// per thread) only while their shared memory, in the single-code-buffer layout, still
+// leaves two CTAs per SM (measured: FP64 n = 192 +12 %, FP32 n = 256 +43 %; FP64 n = 256
+// with the round-1 layout needed one CTA per SM and was 20 % slower with tables, with
+// the aliased single-buffer layout it fits two and is 4 % faster than without tables at
+// three CTAs per SM -- profiles/r02_tables_n256_ab.txt)
 #ifndef MPCGS_PT_SMEM_MAX
 #define MPCGS_PT_SMEM_MAX (110 * 1024)
 #endif
@@ -1516,7 +1524,7 @@ template <typename T, bool GM>
 inline bool product_tables(int n) {
     if (n <= 128) return true;
     if (n > 256) return false;
-    return tab_smem_bytes<T, PRUNE_DR, PRUNE_SI_LARGE, true, GM>(n - 1, std::min(8, PRUNE_DR + PRUNE_SPILL), 0) <=
+    return tab_smem_bytes<T, PRUNE_DR, PRUNE_SI_LARGE, true, GM>(n - 1, std::min(8, PRUNE_DR + PRUNE_SPILL), 0, 1) <=
            (size_t)MPCGS_PT_SMEM_MAX;
 }
 
