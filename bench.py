@@ -476,6 +476,18 @@ def main():
             "prune_share_of_step": prune_ms / loop_ms,
             "partials_per_s_prune_only": N * L * (n - 1) / (prune_avg_s * world) if world == 1 else
             local_trees * L * (n - 1) / prune_avg_s}
+    pp = roof.get("pipe") or {}
+    if pp.get("shared_wavefront_pct") is not None:
+        # the three candidate units side by side, the binding one named
+        units = {"fp_pipe_pct": pp.get("fp64_pipe_active_pct") if args.precision == 64 else pp.get("fma_pipe_active_pct"),
+                 "shared_pipe_pct": pp.get("shared_wavefront_pct"),
+                 "issue_pct": pp.get("issue_active_pct"),
+                 "dram_pct": 100.0 * (pp.get("dram_bytes") or 0.0) / (pp["ncu_duration_ms"] * 1e-3) / 1e9 /
+                             float(mp.get("hbm_gbs", 6540.8)) if pp.get("ncu_duration_ms") else None}
+        top = max((k for k in units if units[k] is not None), key=lambda k: units[k])
+        roof["units"] = units
+        roof["binding"] = (f"latency-bound issue ({pp.get('warps_active_pct', 0):.0f} % of warp slots active); "
+                           f"most utilised unit: {top.replace('_pct', '')} {units[top]:.0f} %")
     if args.compress:
         roof["traffic"] = None  # the ncu traffic on file is the uncompressed launch's
         roof["scored_sites"] = L_scored

@@ -1768,6 +1768,13 @@ mpcgs_status mpcgs_load_state(mpcgs_ctx* c, const void* buf, size_t bytes) {
     std::memcpy(age.data(), p + 16 * nn, 8 * nn);
     std::string why;
     if (check_tree(c->n, parent.data(), age.data(), why)) return fail(c, MPCGS_E_ARG, "load_state: " + why);
+    {
+        std::vector<int32_t> need(nn);
+        std::memcpy(need.data(), p + 12 * nn, 4 * nn);
+        for (size_t v = 0; v < nn; ++v)
+            if (parent[v] < 0 && need[v] > c->depth)
+                return fail(c, MPCGS_E_ARG, "load_state: tree needs more registers than compiled");
+    }
     mpcgs_status st = enter(c);
     if (st) return st;
     for (int32_t* a : {c->s.parent, c->s.left, c->s.right, c->s.need}) {

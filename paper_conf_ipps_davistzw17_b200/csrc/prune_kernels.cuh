@@ -855,6 +855,9 @@ __host__ __device__ constexpr size_t align16(size_t x) { return (x + 15) & ~(siz
 #ifndef MPCGS_SINGLEBUF
 #define MPCGS_SINGLEBUF 1
 #endif
+#ifndef MPCGS_GM32_MAXCTA
+#define MPCGS_GM32_MAXCTA 4
+#endif
 template <typename T, int DR, int SI, bool PT, bool GM = false, int BITS = 2>
 struct TabLayout {
     size_t e, tab, opc, cod, bufb, spill, d, tl, pos, total;
@@ -1465,8 +1468,12 @@ static int tab_trip_cap(K kern, int nops, int need_cap, int& bufs) {
             base = base1;
             blocks = blocks1;
         }
-#ifdef MPCGS_GM32_MAXCTA  // tuning: occupancy cap of the FP32 general-model kernel (room for triplets)
+        // FP32 general model (96 registers, 5 CTAs/SM by registers): the triplet tables the
+        // room at 4 CTAs/SM buys are worth more than the fifth CTA (c5 F84 5.77 -> 5.27 ms,
+        // profiles/r02_gm32_occupancy_ab.txt)
         if (GM && sizeof(T) == 4) blocks = std::min(blocks, MPCGS_GM32_MAXCTA);
+#ifdef MPCGS_F81_32_MAXCTA  // tuning: the same cap for the FP32 F81 kernel
+        if (!GM && sizeof(T) == 4) blocks = std::min(blocks, MPCGS_F81_32_MAXCTA);
 #endif
         if (PT && !MPCGS_NO_TRIPLETS && blocks > 0) {
             const long room = std::min<long>(optin, per_sm / blocks - resv - 256) - (long)fa.sharedSizeBytes - (long)base;
