@@ -564,10 +564,18 @@ __host__ __device__ constexpr bool sparse_checks() { return MPCGS_SPARSE && size
 #ifndef MPCGS_UNITBR
 #define MPCGS_UNITBR 1
 #endif
+#ifndef MPCGS_UNITBR32
+#define MPCGS_UNITBR32 0  // FP32: measured -8 % at c5 (the second loop instance costs the issue-bound
+                          // FP32 kernel more than the FMUL it saves; profiles/r02_kernel_iterations.md)
+#endif
 template <typename T, bool GM>
 __host__ __device__ constexpr bool unit_branch() {
-    return MPCGS_UNITBR && !GM && sizeof(T) == 8;
+    return MPCGS_UNITBR && !GM && (sizeof(T) == 8 || MPCGS_UNITBR32);
 }
+// the unit form's growth budget in bits: a standard-form vector is < 2^(n-1) after
+// power-of-two rescales, and the unit form multiplies it by at most 2^(-C / ln 2)
+template <typename T>
+__host__ __device__ constexpr int unit_budget_bits() { return sizeof(T) == 8 ? 900 : 120; }
 
 template <typename T>
 struct Bounds;
@@ -990,7 +998,7 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
     // and the root 1 / prod_b e_b, the same at every site: ln L_s = ln(pi . root_s) +
     // scale_s ln 2 + C with C = sum_b ln e_b = -u (tree length), added once per tree
     // (exact_commit).  Those factors only enlarge vectors (the S5 lower bounds stay
-    // valid); the form is used while they cannot overflow: -C / ln 2 <= 900 - n bits
+    // valid); the form is used while they cannot overflow: -C / ln 2 <= 900 - n bits (FP32: 120 - n)
     // (a vector of the standard form is < 2^(n-1) after power-of-two rescales), else
     // the tree keeps the standard branch.  C is reduced in a fixed order, so every CTA
     // of a tree (any tiling, any world size) adds the same double (P22).
@@ -1005,11 +1013,15 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
         lnC = s_lne[0];
 #pragma unroll
         for (int w = 1; w < PRUNE_THREADS / 32; ++w) lnC += s_lne[w];
-        unit = -lnC * 1.4426950408889634 <= (double)(900 - n);  // false for -inf / NaN
+        unit = -lnC * 1.4426950408889634 <= (double)(unit_budget_bits<T>() - n);  // false for -inf / NaN
         if (unit) {
             for (int i = tid; i < nops; i += PRUNE_THREADS) {
-                const E4 ed = s_e[i];
-                s_e[i] = make_double4(1.0, ed.y / ed.x, 1.0, ed.w / ed.z);  // {1, r = em / e} per side
+                E4 ed = s_e[i];
+                ed.y = ed.y / ed.x;  // {1, r = em / e} per side
+                ed.w = ed.w / ed.z;
+                ed.x = (T)1;
+                ed.z = (T)1;
+                s_e[i] = ed;
             }
         } else {
             lnC = 0.0;
