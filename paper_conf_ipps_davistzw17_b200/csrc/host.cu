@@ -705,12 +705,19 @@ void incr_tiling(int n, int L, int ntrees_global, int precision, int& tiles, int
     tiles = (L + sites_per_cta - 1) / sites_per_cta;
 }
 
+#ifndef MPCGS_UNIT_MIN_L
+#define MPCGS_UNIT_MIN_L 16384
+#endif
 PruneArgs prune_args(mpcgs_ctx* c, int ntrees, double* out, int out_first, int out_stride) {
     PruneArgs a{};
     a.codes = c->s.codes;
     a.codes2 = c->codes2;
     a.site_w = c->s.site_w;
     a.sum_w = (double)c->L_orig;  // pattern counts sum to the alignment's columns
+    // unit-diagonal branches only on long alignments: their per-CTA setup (a log per branch,
+    // one more barrier) is paid back over many batches (c5 L = 1e5 +1 %, L <= 3 kbp -1..-3.5 %).
+    // A function of the alignment only, so every tiling / world size scores a tree the same way
+    a.unit_form = c->L >= MPCGS_UNIT_MIN_L;
     a.W2 = codes2_words(c->L) * (c->s.amb ? 2 : 1);  // 4-bit codes with ambiguity data
     a.Lpad = c->Lpad;
     a.L = c->L;

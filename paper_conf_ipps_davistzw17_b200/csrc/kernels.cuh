@@ -36,6 +36,7 @@ struct PruneArgs {
     int tiles, sites_per_cta, units, unit_sites;
     const double* site_w;      // [L] pattern counts (compressed sites, f3) or nullptr
     double sum_w;              // sum of the site weights (= alignment columns)
+    int unit_form;             // FP64 table kernel: unit-diagonal branches allowed (a function of the alignment only)
     const int32_t* tree_need;  // [ntrees] register need of each tree's schedule (nullable)
     int need_cap;              // set by launch_prune: largest need the table kernel serves
     int trip_cap;              // set by launch_prune: fused triplets per tree (table kernel)

@@ -928,7 +928,7 @@ static __device__ long long g_pts[8];
 // One CTA scores genealogy `tree` over site tile `tile`; its schedule is gop / ge
 // (global memory written by k_propose); smem_raw = the
 // dynamic shared memory of tab_smem_bytes.
-template <typename T, int DR, int SI, bool PT, int DMX, bool W, bool GM, int BITS>
+template <typename T, int DR, int SI, bool PT, int DMX, bool W, bool GM, int BITS, bool UK>
 __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int tile, const uint32_t* gop,
                                                const typename Traits<T>::E4* ge, unsigned char* smem_raw) {
     using E4 = typename Traits<T>::E4;
@@ -990,7 +990,8 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
             const int lp = Bounds<T>::ilogb(pimin);
             s_d[2 * i] = Bounds<T>::ilogb((T)ed.y) + lp;
             s_d[2 * i + 1] = Bounds<T>::ilogb((T)ed.w) + lp;
-            if constexpr (unit_branch<T, GM>()) lne += log((double)ed.x) + log((double)ed.z);
+            if constexpr (UK && unit_branch<T, GM>())
+                if (a.unit_form) lne += log((double)ed.x) + log((double)ed.z);
         }
     }
     // Unit-diagonal branches (F81, FP64): every branch b of the tree is applied divided
@@ -1004,7 +1005,7 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
     // of a tree (any tiling, any world size) adds the same double (P22).
     bool unit = false;
     double lnC = 0.0;
-    if constexpr (unit_branch<T, GM>()) {
+    if constexpr (UK && unit_branch<T, GM>()) if (a.unit_form) {
         __shared__ double s_lne[PRUNE_THREADS / 32];
 #pragma unroll
         for (int o = 16; o > 0; o >>= 1) lne += __shfl_down_sync(0xffffffffu, lne, o);
@@ -1393,7 +1394,7 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
         acc.reset();
     }
     };
-    if constexpr (unit_branch<T, GM>()) {
+    if constexpr (UK && unit_branch<T, GM>()) {
         if (unit) batches(std::true_type{});
         else batches(std::false_type{});
     } else {
@@ -1412,12 +1413,12 @@ __device__ __forceinline__ void prune_tab_body(const PruneArgs& a, int tree, int
 #endif
 }
 
-template <typename T, int DR, int SI, bool PT, int DMX, bool W, bool GM, int BITS>
+template <typename T, int DR, int SI, bool PT, int DMX, bool W, bool GM, int BITS, bool UK>
 __global__ void MPCGS_TAB_BOUNDS k_prune_tab(PruneArgs a) {
     extern __shared__ __align__(16) unsigned char smem_raw[];
     const int tree = blockIdx.y;
     if (a.tree_need && a.tree_need[tree] > a.need_cap) return;  // deeper tree: scored by the flat pass
-    prune_tab_body<T, DR, SI, PT, DMX, W, GM, BITS>(
+    prune_tab_body<T, DR, SI, PT, DMX, W, GM, BITS, UK>(
         a, tree, blockIdx.x, a.sched_op + (size_t)tree * a.nops,
         reinterpret_cast<const typename Traits<T>::E4*>(a.sched_e) + (size_t)tree * a.nops, smem_raw);
 }
@@ -1503,9 +1504,9 @@ static int tab_trip_cap(K kern, int nops, int need_cap, int& bufs) {
     return cap;
 }
 
-template <typename T, int DR, int SI, bool PT, int DMX, bool W, bool GM, int BITS>
+template <typename T, int DR, int SI, bool PT, int DMX, bool W, bool GM, int BITS, bool UK>
 static cudaError_t launch_tab_w(PruneArgs a, int ntrees, cudaStream_t st) {
-    auto kern = k_prune_tab<T, DR, SI, PT, DMX, W, GM, BITS>;
+    auto kern = k_prune_tab<T, DR, SI, PT, DMX, W, GM, BITS, UK>;
     a.trip_cap = tab_trip_cap<T, DR, SI, PT, GM, BITS>(kern, a.nops, a.need_cap, a.code_bufs);
     const size_t smem = tab_smem_bytes<T, DR, SI, PT, GM, BITS>(a.nops, a.need_cap, a.trip_cap, a.code_bufs);
     static size_t attr_bytes = 48 * 1024;
@@ -1519,10 +1520,10 @@ static cudaError_t launch_tab_w(PruneArgs a, int ntrees, cudaStream_t st) {
     return cudaGetLastError();
 }
 
-template <typename T, int DR, int SI, bool PT, int DMX, bool GM, int BITS>
+template <typename T, int DR, int SI, bool PT, int DMX, bool GM, int BITS, bool UK>
 static cudaError_t launch_tab(const PruneArgs& a, int ntrees, cudaStream_t st) {
-    return a.site_w ? launch_tab_w<T, DR, SI, PT, DMX, true, GM, BITS>(a, ntrees, st)
-                    : launch_tab_w<T, DR, SI, PT, DMX, false, GM, BITS>(a, ntrees, st);
+    return a.site_w ? launch_tab_w<T, DR, SI, PT, DMX, true, GM, BITS, UK>(a, ntrees, st)
+                    : launch_tab_w<T, DR, SI, PT, DMX, false, GM, BITS, UK>(a, ntrees, st);
 }
 
 constexpr int PRUNE_SI_LARGE = 2;  // sites per thread for n > 128
@@ -1547,13 +1548,13 @@ inline bool product_tables(int n) {
            (size_t)MPCGS_PT_SMEM_MAX;
 }
 
-template <typename T, int SI, bool PT, bool GM, int BITS = 2>
+template <typename T, int SI, bool PT, bool GM, int BITS = 2, bool UK = false>
 static cudaError_t launch_tab_dmx(const PruneArgs& a, int ntrees, cudaStream_t st) {
     switch (a.need_cap) {
-        case 1: case 2: case 3: case 4: return launch_tab<T, PRUNE_DR, SI, PT, 4, GM, BITS>(a, ntrees, st);
-        case 5: case 6: return launch_tab<T, PRUNE_DR, SI, PT, 6, GM, BITS>(a, ntrees, st);
-        case 7: case 8: return launch_tab<T, PRUNE_DR, SI, PT, 8, GM, BITS>(a, ntrees, st);
-        default: return launch_tab<T, PRUNE_DR, SI, PT, 10, GM, BITS>(a, ntrees, st);
+        case 1: case 2: case 3: case 4: return launch_tab<T, PRUNE_DR, SI, PT, 4, GM, BITS, UK>(a, ntrees, st);
+        case 5: case 6: return launch_tab<T, PRUNE_DR, SI, PT, 6, GM, BITS, UK>(a, ntrees, st);
+        case 7: case 8: return launch_tab<T, PRUNE_DR, SI, PT, 8, GM, BITS, UK>(a, ntrees, st);
+        default: return launch_tab<T, PRUNE_DR, SI, PT, 10, GM, BITS, UK>(a, ntrees, st);
     }
 }
 
@@ -1566,6 +1567,9 @@ static cudaError_t launch_flat_depth(const PruneArgs& a, int ntrees, int depth, 
         default: return launch_flat<T, 10, GM>(a, ntrees, st);
     }
 }
+
+// FP64 F81 table kernels with the unit-diagonal branch loop (prune_f64_unit.cu)
+cudaError_t launch_tab_unit_f64(const PruneArgs& a, int ntrees, cudaStream_t st);
 
 // one precision x model: instantiated in prune_{f64,f32}{,_gm}.cu (compiled in parallel)
 template <typename T, bool GM>
@@ -1594,7 +1598,12 @@ cudaError_t launch_prune_typed(PruneArgs a, int ntrees, int depth, cudaStream_t 
     const bool deep = prune_max_need(n) > a.need_cap && a.tree_need != nullptr;
     if (!deep) a.tree_need = nullptr;
     const bool pt = !a.amb && product_tables<T, GM>(n);
-    cudaError_t e = a.amb ? (wide_sites(n) ? launch_tab_dmx<T, SI, false, GM, 4>(a, ntrees, st)
+    // FP64 F81 on long alignments (a.unit_form): the kernel with the unit-diagonal
+    // branch loop, a separate instantiation (prune_f64_unit.cu) -- its second loop
+    // instance costs the short-alignment launches 5-9 % (profiles/r02_unit_short_ab.txt)
+    const bool unit_kernel = sizeof(T) == 8 && !GM && MPCGS_UNITBR && a.unit_form && !a.amb && pt && wide_sites(n);
+    cudaError_t e = unit_kernel ? launch_tab_unit_f64(a, ntrees, st)
+                    : a.amb ? (wide_sites(n) ? launch_tab_dmx<T, SI, false, GM, 4>(a, ntrees, st)
                                            : launch_tab_dmx<T, PRUNE_SI_LARGE, false, GM, 4>(a, ntrees, st))
                     : (pt && !wide_sites(n)) ? launch_tab_dmx<T, PRUNE_SI_LARGE, true, GM>(a, ntrees, st)
                     : pt ? launch_tab_dmx<T, SI, true, GM>(a, ntrees, st)

@@ -169,7 +169,7 @@ def test_unit_branch_form_budget(P, orc, n, precision):
     just below and just above the budget (and far above it) must all match the
     oracle, as must short-branch trees (unit form, tiny C)."""
     rng = np.random.default_rng(17 + n)
-    L = 700
+    L = 16400  # the unit form is used on alignments of >= 16384 sites (MPCGS_UNIT_MIN_L)
     pi = np.array([0.2, 0.3, 0.3, 0.2])
     u = orc.default_rate(pi)
     codes = synth.random_alignment(n, L, rng, pi)
